@@ -1,0 +1,260 @@
+"""chgen — seeded synthetic CH-benCHmark / TPC-C table generator.
+
+This module is INPUT ONLY: it produces the column arrays that both the CPU
+oracle (``oracle/``) and the CUDA path (``paper_conf_cidr_appuswamykpa17_b200``)
+consume. It contains none of the queries' arithmetic (no filter, join,
+aggregate or sort of the CH queries) — the two sides share nothing else.
+
+Population follows TPC-C §4.3.3.1 as restated in SURVEY.md Appendix A.3
+([EXT]: the paper itself, PAPER.md, evaluates TPC-H Q6 on lineitem, L687-688,
+and never defines the CH tables). Two modes (reading R9 / SURVEY B9):
+
+* ``strict`` — TPC-C population: delivered lines (o_id < 2101) carry
+  delivery_d = o_entry_d = LOAD_TS, quantity 5, amount 0.00; undelivered lines
+  have delivery NULL and amount U[0.01, 9999.99].
+* ``spread`` — the default for parity and perf: o_entry_d uniform in
+  [1995-01-01, 2025-01-01), delivery_d = o_entry_d + U[0, 30 d) for delivered
+  lines, quantity U[1, 10], amount U[0.01, 9999.99] for every line.
+
+Encodings (R4-R6): ids int32; timestamps int64 µs
+since 1970-01-01 UTC with SQL NULL stored as INT64_MIN; money int64 cents;
+o_carrier_id NULL stored as -1; c_last an int32 dictionary code 0..999.
+
+Every warehouse w draws from its own stream ``Philox(key=[seed, w])`` (item
+uses w = 0), so any warehouse range [a, b) reproduces byte-identical rows to
+the same slice of a full generation — the basis of sharding across ranks.
+"""
+from __future__ import annotations
+
+import datetime as _dt
+from dataclasses import dataclass, field
+
+import numpy as np
+
+__all__ = [
+    "Scale", "TINY", "FULL", "NULL_TS", "LOAD_TS", "TS_1995", "TS_2025",
+    "DAY_US", "ts_us", "generate", "generate_item", "neworder_delta",
+    "warehouse_ranges", "concat_tables", "TABLE_COLUMNS",
+]
+
+
+def ts_us(iso: str) -> int:
+    """int64 µs since the Unix epoch (UTC) of an ISO date/time string."""
+    t = _dt.datetime.fromisoformat(iso).replace(tzinfo=_dt.timezone.utc)
+    return int(t.timestamp()) * 1_000_000
+
+
+NULL_TS = np.iinfo(np.int64).min          # SQL NULL for ol_delivery_d
+LOAD_TS = ts_us("2015-01-01")             # strict-mode o_entry_d
+TS_1995 = ts_us("1995-01-01")
+TS_2025 = ts_us("2025-01-01")
+DAY_US = 86_400 * 1_000_000
+NURAND_C_LAST = 157                       # TPC-C run-time constant C for NURand(255,0,999)
+
+# Column order of each table as the generator emits it (SoA, one ndarray each).
+TABLE_COLUMNS = {
+    "order_line": [("ol_w_id", np.int32), ("ol_d_id", np.int32), ("ol_o_id", np.int32),
+                   ("ol_number", np.int32), ("ol_i_id", np.int32), ("ol_supply_w_id", np.int32),
+                   ("ol_delivery_d", np.int64), ("ol_quantity", np.int32), ("ol_amount", np.int64)],
+    "orders": [("o_w_id", np.int32), ("o_d_id", np.int32), ("o_id", np.int32),
+               ("o_c_id", np.int32), ("o_ol_cnt", np.int32), ("o_carrier_id", np.int32),
+               ("o_all_local", np.int32), ("o_entry_d", np.int64)],
+    "customer": [("c_w_id", np.int32), ("c_d_id", np.int32), ("c_id", np.int32),
+                 ("c_last", np.int32)],
+    "item": [("i_id", np.int32), ("i_price", np.int64)],
+}
+
+
+@dataclass(frozen=True)
+class Scale:
+    """Per-warehouse cardinalities. FULL is TPC-C; TINY is for brute force."""
+    districts: int = 10
+    orders_per_district: int = 3000
+    customers_per_district: int = 3000
+    items: int = 100_000
+    min_ol_cnt: int = 5
+    max_ol_cnt: int = 15
+
+    @property
+    def delivered_below(self) -> int:
+        """o_id threshold for delivered orders: 2101 at 3000 orders (TPC-C)."""
+        return self.orders_per_district * 7 // 10 + 1
+
+
+FULL = Scale()
+TINY = Scale(districts=2, orders_per_district=20, customers_per_district=20, items=100)
+
+
+def _rng(seed: int, w: int) -> np.random.Generator:
+    return np.random.Generator(np.random.Philox(key=np.array([seed, w], dtype=np.uint64)))
+
+
+def _warehouse(w: int, seed: int, mode: str, sc: Scale):
+    if mode not in ("strict", "spread"):
+        raise ValueError(f"mode must be 'strict' or 'spread', not {mode!r}")
+    if sc.orders_per_district > sc.customers_per_district:
+        raise ValueError("o_c_id is a permutation of customers: need orders <= customers")
+    rng = _rng(seed, w)
+    D, O, C = sc.districts, sc.orders_per_district, sc.customers_per_district
+    n_o = D * O
+
+    # ---- orders (PK order: d, o_id) ------------------------------------
+    o_d = np.repeat(np.arange(1, D + 1, dtype=np.int32), O)
+    o_id = np.tile(np.arange(1, O + 1, dtype=np.int32), D)
+    perm = rng.permuted(np.tile(np.arange(1, C + 1, dtype=np.int32), (D, 1)), axis=1)
+    o_c_id = np.ascontiguousarray(perm[:, :O]).reshape(-1)
+    o_ol_cnt = rng.integers(sc.min_ol_cnt, sc.max_ol_cnt + 1, size=n_o, dtype=np.int32)
+    carrier = rng.integers(1, 11, size=n_o, dtype=np.int32)
+    delivered = o_id < sc.delivered_below
+    o_carrier = np.where(delivered, carrier, np.int32(-1)).astype(np.int32)
+    if mode == "strict":
+        o_entry = np.full(n_o, LOAD_TS, dtype=np.int64)
+    else:
+        o_entry = rng.integers(TS_1995, TS_2025, size=n_o, dtype=np.int64)
+
+    # ---- order_line (PK order: d, o_id, ol_number) ----------------------
+    n_ol = int(o_ol_cnt.sum())
+    starts = np.zeros(n_o, dtype=np.int64)
+    np.cumsum(o_ol_cnt[:-1], out=starts[1:])
+    ol_o = np.repeat(o_id, o_ol_cnt)
+    ol_d = np.repeat(o_d, o_ol_cnt)
+    ol_number = (np.arange(n_ol, dtype=np.int64) - np.repeat(starts, o_ol_cnt) + 1).astype(np.int32)
+    ol_i_id = rng.integers(1, sc.items + 1, size=n_ol, dtype=np.int32)
+    ol_deliv_mask = np.repeat(delivered, o_ol_cnt)
+    ol_entry = np.repeat(o_entry, o_ol_cnt)
+    if mode == "strict":
+        ol_delivery = np.where(ol_deliv_mask, ol_entry, NULL_TS)
+        ol_qty = np.full(n_ol, 5, dtype=np.int32)
+        amt = rng.integers(1, 1_000_000, size=n_ol, dtype=np.int64)
+        ol_amount = np.where(ol_deliv_mask, np.int64(0), amt)
+    else:
+        lag = rng.integers(0, 30 * DAY_US, size=n_ol, dtype=np.int64)
+        ol_delivery = np.where(ol_deliv_mask, ol_entry + lag, NULL_TS)
+        ol_qty = rng.integers(1, 11, size=n_ol, dtype=np.int32)
+        ol_amount = rng.integers(1, 1_000_000, size=n_ol, dtype=np.int64)
+
+    # ---- customer (PK order: d, c_id) -----------------------------------
+    c_d = np.repeat(np.arange(1, D + 1, dtype=np.int32), C)
+    c_id = np.tile(np.arange(1, C + 1, dtype=np.int32), D)
+    a = rng.integers(0, 256, size=D * C, dtype=np.int32)
+    b = rng.integers(0, 1000, size=D * C, dtype=np.int32)
+    nurand = ((a | b) + NURAND_C_LAST) % 1000
+    c_last = np.where(c_id <= 1000, c_id - 1, nurand).astype(np.int32)
+
+    wi = np.int32(w)
+    ol = {
+        "ol_w_id": np.full(n_ol, wi, dtype=np.int32), "ol_d_id": ol_d, "ol_o_id": ol_o,
+        "ol_number": ol_number, "ol_i_id": ol_i_id,
+        "ol_supply_w_id": np.full(n_ol, wi, dtype=np.int32),
+        "ol_delivery_d": ol_delivery.astype(np.int64), "ol_quantity": ol_qty.astype(np.int32),
+        "ol_amount": ol_amount.astype(np.int64),
+    }
+    orders = {
+        "o_w_id": np.full(n_o, wi, dtype=np.int32), "o_d_id": o_d, "o_id": o_id,
+        "o_c_id": o_c_id, "o_ol_cnt": o_ol_cnt, "o_carrier_id": o_carrier,
+        "o_all_local": np.ones(n_o, dtype=np.int32), "o_entry_d": o_entry,
+    }
+    customer = {"c_w_id": np.full(D * C, wi, dtype=np.int32), "c_d_id": c_d, "c_id": c_id,
+                "c_last": c_last}
+    return {"order_line": ol, "orders": orders, "customer": customer}
+
+
+def generate_item(seed: int = 1, scale: Scale = FULL):
+    """item table (replicated on every rank), stream key [seed, 0]."""
+    rng = _rng(seed, 0)
+    return {"i_id": np.arange(1, scale.items + 1, dtype=np.int32),
+            "i_price": rng.integers(100, 10_001, size=scale.items, dtype=np.int64)}
+
+
+def concat_tables(parts):
+    """Concatenate a list of {table: {col: array}} dicts table by table."""
+    out = {}
+    for t in parts[0]:
+        out[t] = {c: np.concatenate([p[t][c] for p in parts]) for c in parts[0][t]}
+    return out
+
+
+def generate(w_lo: int, w_hi: int | None = None, *, seed: int = 1, mode: str = "spread",
+             scale: Scale = FULL, with_item: bool = True):
+    """Tables for warehouses [w_lo, w_hi) (1-based ids). ``generate(1, W+1)`` is W warehouses.
+
+    Returns ``{"order_line": {...}, "orders": {...}, "customer": {...}, "item": {...}}``
+    with each column a contiguous numpy array in the dtype of TABLE_COLUMNS.
+    """
+    if w_hi is None:
+        w_lo, w_hi = 1, w_lo + 1
+    if not (1 <= w_lo <= w_hi):
+        raise ValueError("warehouse ids are 1-based and w_lo <= w_hi")
+    if w_hi == w_lo:
+        empty = {t: {c: np.zeros(0, dtype=dt) for c, dt in cols}
+                 for t, cols in TABLE_COLUMNS.items() if t != "item"}
+        parts = [empty]
+    else:
+        parts = [_warehouse(w, seed, mode, scale) for w in range(w_lo, w_hi)]
+    out = concat_tables(parts) if len(parts) > 1 else parts[0]
+    if with_item:
+        out["item"] = generate_item(seed, scale)
+    return out
+
+
+def warehouse_ranges(n_warehouses: int, world: int):
+    """Contiguous warehouse ranges [lo, hi) per rank (R15)."""
+    base, extra = divmod(n_warehouses, world)
+    out, lo = [], 1
+    for r in range(world):
+        hi = lo + base + (1 if r < extra else 0)
+        out.append((lo, hi))
+        lo = hi
+    return out
+
+
+@dataclass
+class NewOrderState:
+    """Per-district next o_id for appended NewOrder transactions (config C5 input)."""
+    w_lo: int
+    w_hi: int
+    scale: Scale = FULL
+    next_o_id: dict = field(default_factory=dict)
+    clock: int = TS_2025
+
+
+def neworder_delta(state: NewOrderState, n_txn: int, *, seed: int, batch: int,
+                   item=None):
+    """Rows appended by ``n_txn`` TPC-C NewOrder transactions.
+
+    Simplified TPC-C 2.4.1 input generation: district uniform, customer uniform,
+    ol_cnt U[5,15], item uniform, qty U[1,10], amount = qty * i_price, delivery NULL,
+    o_entry_d a logical clock starting 2025-01-01. No rollbacks in this delta.
+    Returns ``{"order_line": {...}, "orders": {...}}`` for the appended rows only.
+    """
+    sc = state.scale
+    rng = np.random.Generator(np.random.Philox(key=np.array([seed, 1 << 40 | batch], dtype=np.uint64)))
+    if item is None:
+        item = generate_item(seed, sc)
+    cols_o = {c: [] for c, _ in TABLE_COLUMNS["orders"]}
+    cols_l = {c: [] for c, _ in TABLE_COLUMNS["order_line"]}
+    for _ in range(n_txn):
+        w = int(rng.integers(state.w_lo, state.w_hi))
+        d = int(rng.integers(1, sc.districts + 1))
+        key = (w, d)
+        o = state.next_o_id.get(key, sc.orders_per_district + 1)
+        state.next_o_id[key] = o + 1
+        c = int(rng.integers(1, sc.customers_per_district + 1))
+        cnt = int(rng.integers(sc.min_ol_cnt, sc.max_ol_cnt + 1))
+        state.clock += 1_000
+        for k, v in (("o_w_id", w), ("o_d_id", d), ("o_id", o), ("o_c_id", c),
+                     ("o_ol_cnt", cnt), ("o_carrier_id", -1), ("o_all_local", 1),
+                     ("o_entry_d", state.clock)):
+            cols_o[k].append(v)
+        iids = rng.integers(1, sc.items + 1, size=cnt)
+        qtys = rng.integers(1, 11, size=cnt)
+        for n in range(cnt):
+            i = int(iids[n])
+            q = int(qtys[n])
+            for k, v in (("ol_w_id", w), ("ol_d_id", d), ("ol_o_id", o), ("ol_number", n + 1),
+                         ("ol_i_id", i), ("ol_supply_w_id", w), ("ol_delivery_d", int(NULL_TS)),
+                         ("ol_quantity", q), ("ol_amount", q * int(item["i_price"][i - 1]))):
+                cols_l[k].append(v)
+    dts = {c: dt for t in ("orders", "order_line") for c, dt in TABLE_COLUMNS[t]}
+    return {"orders": {k: np.asarray(v, dtype=dts[k]) for k, v in cols_o.items()},
+            "order_line": {k: np.asarray(v, dtype=dts[k]) for k, v in cols_l.items()}}

@@ -1,0 +1,159 @@
+"""CPU oracle for CH-benCHmark Q1 / Q6 / Q18 — TEST INFRASTRUCTURE ONLY.
+
+Only ``tests/``, ``__graft_entry__.smoke()`` and ``bench.py`` (its ``cpu_baseline``
+leg and ``--impl reference``) may import this package. The product path
+(``paper_conf_cidr_appuswamykpa17_b200``) never imports it and shares no code with it.
+
+The arithmetic lives in ``oracle.c`` (plain C, single-threaded, row at a time, SQL
+three-valued logic; see its header for the passages followed). This module only
+compiles it with gcc and marshals numpy arrays through ctypes.
+
+Pins (tests/test_oracle_*.py): SQLite executing the literal CH SQL; brute-force nested
+loops over the cartesian product on tiny tables; strict-mode closed forms; a
+hand-derived golden fixture (tests/golden/); re-partition and COUNT invariants.
+"""
+from __future__ import annotations
+
+import ctypes as C
+import os
+import subprocess
+
+import numpy as np
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+_SRC = os.path.join(_HERE, "oracle.c")
+_HDR = os.path.join(_HERE, "oracle.h")
+_LIB = os.path.join(_HERE, "liboracle.so")
+
+OR_OVERFLOW = -1
+OR_NOMEM = -2
+
+
+def build(force: bool = False) -> str:
+    """Compile liboracle.so with gcc (-O2, no vectorisation tricks needed)."""
+    stale = (not os.path.exists(_LIB)) or max(os.path.getmtime(_SRC), os.path.getmtime(_HDR)) > os.path.getmtime(_LIB)
+    if force or stale:
+        tmp = _LIB + f".{os.getpid()}.tmp"
+        subprocess.check_call(["gcc", "-O2", "-std=c11", "-Wall", "-Wextra", "-fPIC", "-shared",
+                               "-o", tmp, _SRC])
+        os.replace(tmp, _LIB)
+    return _LIB
+
+
+class _OL(C.Structure):
+    _fields_ = [("n", C.c_int64), ("w_id", C.c_void_p), ("d_id", C.c_void_p), ("o_id", C.c_void_p),
+                ("number", C.c_void_p), ("delivery_d", C.c_void_p), ("quantity", C.c_void_p),
+                ("amount", C.c_void_p)]
+
+
+class _O(C.Structure):
+    _fields_ = [("n", C.c_int64), ("w_id", C.c_void_p), ("d_id", C.c_void_p), ("o_id", C.c_void_p),
+                ("c_id", C.c_void_p), ("ol_cnt", C.c_void_p), ("entry_d", C.c_void_p)]
+
+
+class _C(C.Structure):
+    _fields_ = [("n", C.c_int64), ("w_id", C.c_void_p), ("d_id", C.c_void_p), ("c_id", C.c_void_p),
+                ("c_last", C.c_void_p)]
+
+
+_lib = None
+
+
+def _load():
+    global _lib
+    if _lib is None:
+        lib = C.CDLL(build())
+        lib.oracle_q6.restype = C.c_int
+        lib.oracle_q1.restype = C.c_int64
+        lib.oracle_q18.restype = C.c_int64
+        _lib = lib
+    return _lib
+
+
+def _p(a):
+    return a.ctypes.data_as(C.c_void_p) if a is not None else None
+
+
+def _col(t, name, dtype):
+    a = np.ascontiguousarray(t[name], dtype=dtype)
+    return a
+
+
+class _Keep:
+    """Holds contiguous copies alive for the duration of a call."""
+
+    def __init__(self):
+        self.arrs = []
+
+    def __call__(self, a):
+        self.arrs.append(a)
+        return _p(a)
+
+
+def _ol_struct(ol, keep):
+    n = len(ol["ol_w_id"])
+    return _OL(n, keep(_col(ol, "ol_w_id", np.int32)), keep(_col(ol, "ol_d_id", np.int32)),
+               keep(_col(ol, "ol_o_id", np.int32)), keep(_col(ol, "ol_number", np.int32)),
+               keep(_col(ol, "ol_delivery_d", np.int64)), keep(_col(ol, "ol_quantity", np.int32)),
+               keep(_col(ol, "ol_amount", np.int64)))
+
+
+def _check(st):
+    if st == OR_OVERFLOW:
+        raise OverflowError("integer overflow in SUM (oracle)")
+    if st == OR_NOMEM:
+        raise MemoryError("oracle out of memory")
+
+
+def q6(tables, d_lo, d_hi, q_lo, q_hi):
+    """CH Q6. Returns {"revenue": int or None (NULL), "count": qualifying rows}."""
+    lib, keep = _load(), _Keep()
+    ol = _ol_struct(tables["order_line"], keep)
+    rev, isnull, cnt = C.c_int64(), C.c_int32(), C.c_int64()
+    _check(lib.oracle_q6(C.byref(ol), C.c_int64(d_lo), C.c_int64(d_hi), C.c_int64(q_lo),
+                         C.c_int64(q_hi), C.byref(rev), C.byref(isnull), C.byref(cnt)))
+    return {"revenue": None if isnull.value else rev.value, "count": cnt.value}
+
+
+def q1(tables, cutoff):
+    """CH Q1. Returns a dict of numpy columns ordered by ol_number."""
+    lib, keep = _load(), _Keep()
+    ol = _ol_struct(tables["order_line"], keep)
+    cap = 64
+    while True:
+        out = {"ol_number": np.zeros(cap, np.int32), "sum_qty": np.zeros(cap, np.int64),
+               "sum_amount": np.zeros(cap, np.int64), "avg_qty": np.zeros(cap, np.float64),
+               "avg_amount": np.zeros(cap, np.float64), "count_order": np.zeros(cap, np.int64)}
+        n = lib.oracle_q1(C.byref(ol), C.c_int64(cutoff), C.c_int64(cap),
+                          _p(out["ol_number"]), _p(out["sum_qty"]), _p(out["sum_amount"]),
+                          _p(out["avg_qty"]), _p(out["avg_amount"]), _p(out["count_order"]))
+        _check(n if n < 0 else 0)
+        if n <= cap:
+            return {k: v[:n] for k, v in out.items()}
+        cap = n
+
+
+Q18_COLUMNS = [("c_last", np.int32), ("c_id", np.int32), ("o_id", np.int32), ("o_entry_d", np.int64),
+               ("o_ol_cnt", np.int32), ("amount_sum", np.int64), ("o_w_id", np.int32),
+               ("o_d_id", np.int32)]
+
+
+def q18(tables, having):
+    """CH Q18 (customer ⋈ orders ⋈ order_line). Returns numpy columns in ORDER BY order."""
+    lib, keep = _load(), _Keep()
+    ol = _ol_struct(tables["order_line"], keep)
+    o, c = tables["orders"], tables["customer"]
+    os_ = _O(len(o["o_w_id"]), keep(_col(o, "o_w_id", np.int32)), keep(_col(o, "o_d_id", np.int32)),
+             keep(_col(o, "o_id", np.int32)), keep(_col(o, "o_c_id", np.int32)),
+             keep(_col(o, "o_ol_cnt", np.int32)), keep(_col(o, "o_entry_d", np.int64)))
+    cs = _C(len(c["c_w_id"]), keep(_col(c, "c_w_id", np.int32)), keep(_col(c, "c_d_id", np.int32)),
+            keep(_col(c, "c_id", np.int32)), keep(_col(c, "c_last", np.int32)))
+    cap = max(1, len(o["o_w_id"]))
+    while True:
+        out = {k: np.zeros(cap, dt) for k, dt in Q18_COLUMNS}
+        n = lib.oracle_q18(C.byref(cs), C.byref(os_), C.byref(ol), C.c_int64(having), C.c_int64(cap),
+                           *[_p(out[k]) for k, _ in Q18_COLUMNS])
+        _check(n if n < 0 else 0)
+        if n <= cap:
+            return {k: v[:n] for k, v in out.items()}
+        cap = n

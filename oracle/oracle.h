@@ -1,0 +1,81 @@
+/*
+ * oracle.h — CPU ORACLE for the CH-benCHmark OLAP hot path. TEST INFRASTRUCTURE ONLY.
+ *
+ * Only tests/, __graft_entry__.smoke() and bench.py's cpu_baseline / --impl reference
+ * legs may load liboracle.so. It shares no code, header, table or constant with the
+ * CUDA path (paper_conf_cidr_appuswamykpa17_b200/, include/), and never includes them.
+ *
+ * What it computes: the plain SQL definitions of CH-benCHmark Q1, Q6 and Q18
+ * (SURVEY.md Appendix A.1 [EXT]; the paper's OLAP path is PAPER.md L524-572, its only
+ * query text is "TPC-H Q6, a selection over the lineitem table", L687-688), evaluated
+ * row at a time, single-threaded, with SQL three-valued logic for NULLs.
+ *
+ * Encodings (R4-R6): timestamps int64 µs UTC, NULL = INT64_MIN (decoded here,
+ * independently of the GPU path); money int64 cents; ids/quantities int32.
+ *
+ * Parity pins: tests/test_oracle_*.py — SQLite running the literal CH SQL, brute-force
+ * nested loops on tiny tables, strict-mode closed forms, hand-derived golden fixture
+ * (tests/golden/), re-partition and COUNT invariants. No function here is "parity unpinned".
+ */
+#ifndef H2TAP_ORACLE_H
+#define H2TAP_ORACLE_H
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+/* Borrowed, caller-owned column pointers (SoA). */
+typedef struct {
+    int64_t n;
+    const int32_t *w_id, *d_id, *o_id, *number;
+    const int64_t *delivery_d;      /* INT64_MIN = NULL */
+    const int32_t *quantity;
+    const int64_t *amount;          /* cents */
+} or_order_line;
+
+typedef struct {
+    int64_t n;
+    const int32_t *w_id, *d_id, *o_id, *c_id, *ol_cnt;
+    const int64_t *entry_d;
+} or_orders;
+
+typedef struct {
+    int64_t n;
+    const int32_t *w_id, *d_id, *c_id, *c_last;
+} or_customer;
+
+/* Status codes. */
+#define OR_OK        0
+#define OR_OVERFLOW -1   /* an int64 SUM overflowed (SQLite raises "integer overflow") */
+#define OR_NOMEM    -2
+
+/* CH Q6: SELECT SUM(ol_amount) FROM order_line WHERE ol_delivery_d >= d_lo AND
+ * ol_delivery_d < d_hi AND ol_quantity BETWEEN q_lo AND q_hi.
+ * *revenue_is_null = 1 when no row qualifies (SUM over the empty set is NULL).
+ * *count = number of qualifying rows (not part of the SQL output; used by invariants). */
+int oracle_q6(const or_order_line *ol, int64_t d_lo, int64_t d_hi, int64_t q_lo, int64_t q_hi,
+              int64_t *revenue, int32_t *revenue_is_null, int64_t *count);
+
+/* CH Q1: SELECT ol_number, SUM(ol_quantity), SUM(ol_amount), AVG(ol_quantity),
+ * AVG(ol_amount), COUNT(*) FROM order_line WHERE ol_delivery_d > cutoff
+ * GROUP BY ol_number ORDER BY ol_number.
+ * avg_amount is in currency units: (sum_cents / count) / 100.
+ * Writes min(ngroups, cap) rows; returns ngroups (>= 0) or a negative status. */
+int64_t oracle_q1(const or_order_line *ol, int64_t cutoff, int64_t cap,
+                  int32_t *ol_number, int64_t *sum_qty, int64_t *sum_amount,
+                  double *avg_qty, double *avg_amount, int64_t *count_order);
+
+/* CH Q18 (customer ⋈ orders ⋈ order_line, GROUP BY, HAVING SUM(ol_amount) > having):
+ * output columns c_last, c_id, o_id, o_entry_d, o_ol_cnt, amount_sum, plus o_w_id, o_d_id
+ * (R3), ordered by amount_sum DESC, o_entry_d ASC, then o_w_id, o_d_id, o_id,
+ * c_id, c_last, o_ol_cnt ASC (R11). Writes min(nrows, cap) rows; returns nrows or < 0. */
+int64_t oracle_q18(const or_customer *c, const or_orders *o, const or_order_line *ol,
+                   int64_t having, int64_t cap,
+                   int32_t *c_last, int32_t *c_id, int32_t *o_id, int64_t *o_entry_d,
+                   int32_t *o_ol_cnt, int64_t *amount_sum, int32_t *o_w_id, int32_t *o_d_id);
+
+#ifdef __cplusplus
+}
+#endif
+#endif
