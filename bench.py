@@ -1,0 +1,371 @@
+#!/usr/bin/env python
+"""bench.py — CH-benCHmark OLAP hot path on B200 (H2TAP / Caldera data-parallel archipelago).
+
+One STEP = one pass of the whole hot path over the rank's resident snapshot: CH Q6 (fused
+scan-filter-sum), CH Q1 (fused scan-filter-group-by) and CH Q18 (hash build, probe +
+group-join, HAVING compaction, customer probe, ORDER BY) through the C ABI, each with its
+cross-GPU merge when N > 1. Workload = BASELINE.json configs[1]/[2]: W = 100 TPC-C warehouses
+per GPU (~30M order_line rows), synthetic ('spread' population, seed 1).
+
+value  = order_line rows processed per second by the step's three queries, whole job
+         (3 x visible order_line rows x N / step time), snapshot resident in HBM.
+e2e    = same metric through the public API with host buffers: each step refreshes the snapshot
+         from pinned host memory (full reload, H2D inside the timed region) and returns every
+         result to host memory.
+roofline: the dominant kernel's algorithmic bytes per launch / its CUDA-event duration,
+         against MEASURED_PEAKS.json hbm_gbs.
+
+Usage: python bench.py [--gpus N --steps K --warmup W] [--impl ours|reference]
+       torchrun --nproc-per-node N bench.py --gpus N ...
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import tempfile
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import chgen  # noqa: E402
+
+METRIC = "CH-benCHmark Q1/Q6 order_line rows/s & latency; % of HBM BW, 1/2/4/8 B200"
+UNIT = "order_line rows/s"
+Q6_P = [chgen.ts_us("1999-01-01"), chgen.ts_us("2020-01-01"), 1, 100000]
+Q1_P = [chgen.ts_us("2007-01-02")]
+Q18_P = [20000]
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
+    ap.add_argument("--warehouses", type=int, default=100, help="warehouses per GPU (weak scaling)")
+    ap.add_argument("--mode", default="spread", choices=["spread", "strict"])
+    ap.add_argument("--e2e-steps", type=int, default=None)
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-flush-l2", action="store_true")
+    return ap.parse_args()
+
+
+# ------------------------------------------------------------------ plumbing --
+def dist_env():
+    rank = int(os.environ.get("RANK", "0"))
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    return rank, world, local
+
+
+class Clocks:
+    """nvidia-smi sampling during the timed region (B200_PROFILING.md clocks line)."""
+
+    def __init__(self, index):
+        self.path = tempfile.mktemp(suffix=".csv")
+        q = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,"
+             "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+             "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+        try:
+            self.p = subprocess.Popen(["nvidia-smi", f"--id={index}", f"--query-gpu={q}",
+                                       "--format=csv,noheader,nounits", "-lms", "100"],
+                                      stdout=open(self.path, "w"), stderr=subprocess.DEVNULL)
+        except Exception:
+            self.p = None
+
+    def stop(self):
+        if not self.p:
+            return None
+        self.p.terminate()
+        self.p.wait()
+        sm, mx, reasons = [], 0, set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for line in open(self.path):
+            f = [x.strip() for x in line.split(",")]
+            if len(f) < 9:
+                continue
+            try:
+                sm.append(float(f[1]))
+                mx = max(mx, float(f[2]))
+            except ValueError:
+                continue
+            for n, v in zip(names, f[5:9]):
+                if v.lower() == "active":
+                    reasons.add(n)
+        os.unlink(self.path)
+        if not sm:
+            return None
+        return {"sm_mhz": statistics.median(sm), "sm_max_mhz": mx, "reasons": sorted(reasons),
+                "samples": len(sm)}
+
+
+def peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    if os.path.exists(p):
+        d = json.load(open(p))
+        return float(d["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs: copy, read+write bytes)"
+    return 6650.0, "fallback (B200_PROFILING.md 6.65 TB/s)"
+
+
+def ncu_traffic():
+    """Per-launch DRAM bytes of each kernel from the committed ncu --set full capture."""
+    p = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    if os.path.exists(p):
+        return json.load(open(p))
+    return {}
+
+
+# ------------------------------------------------------------- algorithmic bytes --
+def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes):
+    """Bytes the method must move per launch."""
+    cap_o = 1 << max(4, int(np.ceil(np.log2(max(2 * n_o, 16)))))
+    cap_c = 1 << max(4, int(np.ceil(np.log2(max(2 * n_c, 16)))))
+    return {
+        "q6_scan_filter_sum": 20 * n_ol,
+        "q1_scan_filter_groupby": 24 * n_ol,
+        "q18_init": 16 * (cap_o + cap_c + n_o),
+        "q18_build": 12 * n_o + 12 * n_c + 16 * (n_o + n_c),
+        "q18_probe_groupjoin": 20 * n_ol + 16 * n_o + 16 * n_o,
+        "q18_having_compact": 16 * n_o + 28 * n_o + 16 * n_pass + 4 * n_pass + 40 * n_pass,
+        "q18_sort_keys": 40 * n_pass + 24 * n_pass,
+        "q18_radix_sort": sort_passes * (2 * (4 + 8) + 4 + 4) * n_pass,
+        "q18_permute": (4 + 40 + 40) * n_pass,
+    }.get(kernel)
+
+
+# ------------------------------------------------------------------ reference --
+def cpu_oracle_sample(w_lo, sample_w, mode):
+    """Oracle (single-threaded C, as it stands) on a bounded sample of the same workload."""
+    import oracle
+    t = chgen.generate(w_lo, w_lo + sample_w, seed=1, mode=mode)
+    n = len(t["order_line"]["ol_w_id"])
+    t0 = time.perf_counter()
+    oracle.q6(t, *Q6_P)
+    oracle.q1(t, *Q1_P)
+    oracle.q18(t, *Q18_P)
+    dt = time.perf_counter() - t0
+    return 3 * n / dt, dt, n
+
+
+def run_reference(a):
+    rank, world, _ = dist_env()
+    if rank != 0:
+        return 0
+    import oracle
+    oracle.build()
+    sample_w = 10
+    t = chgen.generate(1, 1 + sample_w, seed=1, mode=a.mode)
+    n = len(t["order_line"]["ol_w_id"])
+    for _ in range(a.warmup):
+        oracle.q6(t, *Q6_P); oracle.q1(t, *Q1_P); oracle.q18(t, *Q18_P)
+    t0 = time.perf_counter()
+    for _ in range(a.steps):
+        oracle.q6(t, *Q6_P); oracle.q1(t, *Q1_P); oracle.q18(t, *Q18_P)
+    dt = time.perf_counter() - t0
+    value = 3 * n * a.steps / dt
+    sample = (f"each step = oracle Q6+Q1+Q18 over W={sample_w} warehouses ({n} order_line rows, "
+              f"'{a.mode}', seed 1), single thread")
+    print(json.dumps({
+        "impl": "reference", "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": a.gpus,
+        "steps": a.steps, "warmup": a.warmup, "ms_per_step": dt / a.steps * 1e3,
+        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "int64",
+        "data": "synthetic", "config": {"workload": f"CH Q6+Q1+Q18 per step, sample W={sample_w}",
+                                        "mode": a.mode},
+        "cpu_baseline": {"value": value, "unit": UNIT, "cores": 1, "kind": "oracle", "sample": sample},
+        "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }))
+    return 0
+
+
+# ----------------------------------------------------------------------- ours --
+def main():
+    a = parse()
+    if a.impl == "reference":
+        return run_reference(a)
+    import torch
+    import torch.distributed as dist
+
+    rank, world, local = dist_env()
+    if world != a.gpus:
+        a.gpus = world if world > 1 else a.gpus
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+
+    import paper_conf_cidr_appuswamykpa17_b200 as h
+
+    # ---- engine + NCCL bootstrap (ncclUniqueId broadcast over the torch process group)
+    nccl_id = None
+    if world > 1:
+        obj = [h.h2tap_nccl_unique_id() if rank == 0 else None]
+        dist.broadcast_object_list(obj, src=0)
+        nccl_id = obj[0]
+    eng = h.h2tap_open(local, rank, world, nccl_id)
+
+    # ---- this rank's warehouse shard (weak scaling: a.warehouses per GPU)
+    W = a.warehouses * world
+    lo, hi = chgen.warehouse_ranges(W, world)[rank]
+    tables = chgen.generate(lo, hi, seed=1, mode=a.mode)
+    hot = h.hot_path_tables(tables)
+    n_ol = len(tables["order_line"]["ol_w_id"])
+    n_o = len(tables["orders"]["o_id"])
+    n_c = len(tables["customer"]["c_id"])
+    pinned = {t: {c: torch.from_numpy(v).pin_memory() for c, v in cols.items()} for t, cols in hot.items()}
+    h2d_bytes = sum(v.numel() * v.element_size() for cols in pinned.values() for v in cols.values())
+    epoch = 1
+    h.h2tap_load_snapshot(eng, pinned, epoch)
+
+    stream = torch.cuda.ExternalStream(h.h2tap_compute_stream(eng))
+    flush = None if a.no_flush_l2 else torch.empty(512 << 20, dtype=torch.uint8, device="cuda")
+
+    def barrier():
+        if world > 1:
+            dist.barrier()
+        torch.cuda.synchronize()
+
+    def step(flags):
+        out = {}
+        for name, plan, p in (("q6", h.H2TAP_Q6, Q6_P), ("q1", h.H2TAP_Q1, Q1_P), ("q18", h.H2TAP_Q18, Q18_P)):
+            r = h.h2tap_run_query(eng, plan, p, flags=flags)
+            out[name] = (r.device_ms, r.kernels, r.nrows, r.kernel_launches)
+            h.h2tap_free(r)
+        return out
+
+    dev_flags = h.H2TAP_RESULT_DEVICE | h.H2TAP_QUERY_PROFILE
+    for _ in range(a.warmup):
+        step(dev_flags)
+    barrier()
+
+    # ---- device-resident timed region: K steps, CUDA events on the engine's stream
+    clocks = Clocks(local)
+    starts = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
+    ends = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
+    per_query = {"q6": [], "q1": [], "q18": []}
+    kern = {}
+    launches = 0
+    n_pass = 0
+    q18_launches = 0
+    barrier()
+    for i in range(a.steps):
+        if flush is not None:
+            with torch.cuda.stream(stream):
+                flush.add_(1)  # write 512 MB > 126 MB L2 between steps, outside the events
+        starts[i].record(stream)
+        out = step(dev_flags)
+        ends[i].record(stream)
+        for q, (ms, ks, nrows, nl) in out.items():
+            per_query[q].append(ms)
+            launches += nl
+            for kname, kms in ks:
+                kern.setdefault(kname, []).append(kms)
+        n_pass = out["q18"][2]
+        q18_launches = out["q18"][3]
+    barrier()
+    clk = clocks.stop()
+    step_ms_local = sum(s.elapsed_time(e) for s, e in zip(starts, ends)) / a.steps
+    t = torch.tensor([step_ms_local], dtype=torch.float64, device="cuda")
+    if world > 1:
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    step_ms = float(t.item())
+    rows_total = 3 * n_ol * world  # weak scaling: every rank holds the same-sized shard
+    value = rows_total / (step_ms / 1e3)
+
+    # ---- roofline for the dominant kernel (largest share of the step)
+    kavg = {k: float(np.mean(v)) for k, v in kern.items()}
+    # radix passes (3 kernels each) are folded into q18_radix_sort; recover the pass count from
+    # the query's launch count: init, build, probe, having, sort_keys, permute + 3 per pass
+    sort_passes = max(0, (q18_launches - 6) // 3)
+    dominant = max(kavg, key=kavg.get) if kavg else None
+    peak, peak_src = peaks()
+    roof = None
+    if dominant:
+        b = alg_bytes(dominant, n_ol, n_o, n_c, n_pass, sort_passes)
+        if b:
+            ach = b / (kavg[dominant] / 1e3) / 1e9
+            tr = ncu_traffic().get(dominant)
+            roof = {"bound": "hbm", "kernel": dominant, "achieved": round(ach, 1), "peak": peak,
+                    "unit": "GB/s", "frac": round(ach / peak, 4), "traffic": tr,
+                    "algorithmic_bytes_per_launch": int(b), "avg_launch_ms": round(kavg[dominant], 5),
+                    "share_of_step": round(kavg[dominant] / step_ms_local, 4), "peak_source": peak_src}
+    kernels_summary = {}
+    for k, v in kavg.items():
+        b = alg_bytes(k, n_ol, n_o, n_c, n_pass, sort_passes)
+        kernels_summary[k] = {"ms": round(v, 5), "share": round(v / step_ms_local, 4)}
+        if b and k != "q18_radix_sort":
+            kernels_summary[k]["GB/s"] = round(b / (v / 1e3) / 1e9, 1)
+            kernels_summary[k]["frac_hbm"] = round(b / (v / 1e3) / 1e9 / peak, 4)
+
+    # ---- e2e: host buffers through the public API (H2D refresh + queries + D2H results)
+    e2e_steps = a.e2e_steps or max(3, min(a.steps, 5))
+    for _ in range(1):  # warm the reload path (spare buffers)
+        epoch += 1
+        h.h2tap_load_snapshot(eng, pinned, epoch)
+        step(0)
+    barrier()
+    d2h = 0
+    t0 = time.perf_counter()
+    for _ in range(e2e_steps):
+        epoch += 1
+        h.h2tap_load_snapshot(eng, pinned, epoch)
+        d2h = 0
+        for plan, p in ((h.H2TAP_Q6, Q6_P), (h.H2TAP_Q1, Q1_P), (h.H2TAP_Q18, Q18_P)):
+            r = h.h2tap_run_query(eng, plan, p)
+            for c in r.columns.values():
+                d2h += c.nbytes
+            _ = r.columns[next(iter(r.columns))][:1].sum() if r.nrows else 0  # host read
+            h.h2tap_free(r)
+    barrier()
+    e2e_s = (time.perf_counter() - t0) / e2e_steps
+    te = torch.tensor([e2e_s], dtype=torch.float64, device="cuda")
+    if world > 1:
+        dist.all_reduce(te, op=dist.ReduceOp.MAX)
+    e2e_s = float(te.item())
+
+    # ---- CPU oracle baseline (rank 0, N = 1 only, bounded sample)
+    cpu = None
+    if rank == 0 and world == 1 and not a.no_cpu_baseline:
+        sample_w = 20
+        v, dt, n = cpu_oracle_sample(lo, sample_w, a.mode)
+        cpu = {"value": v, "unit": UNIT, "cores": 1, "kind": "oracle",
+               "sample": f"oracle Q6+Q1+Q18 once over W={sample_w} of the same warehouses "
+                         f"({n} order_line rows, {dt:.1f} s, single thread)"}
+
+    if rank == 0:
+        line = {
+            "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": a.steps,
+            "warmup": a.warmup, "ms_per_step": step_ms, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "int64", "data": "synthetic",
+            "config": {"workload": f"CH Q6+Q1+Q18 per step over W={a.warehouses} warehouses per GPU "
+                                   f"('{a.mode}' TPC-C population, seed 1)",
+                       "warehouses_per_gpu": a.warehouses, "order_line_rows_per_gpu": n_ol,
+                       "orders_rows_per_gpu": n_o, "customer_rows_per_gpu": n_c,
+                       "queries_per_step": 3, "parallelism": f"row-sharded by warehouse x{world}",
+                       "l2": ("inputs > L2 and 512 MB L2-flush write between steps (outside events)"
+                              if flush is not None else "inputs > L2 (no flush)")},
+            "latency_ms": {q: round(float(np.median(v)), 4) for q, v in per_query.items()},
+            "rows_per_s": {q: n_ol * world / (float(np.median(v)) / 1e3) for q, v in per_query.items()},
+            "q18_result_rows": n_pass,
+            "roofline": roof,
+            "kernels": kernels_summary,
+            "cpu_baseline": cpu,
+            "e2e": {"value": rows_total / e2e_s, "unit": UNIT, "h2d_bytes_per_step": int(h2d_bytes),
+                    "d2h_bytes_per_step": int(d2h), "ms_per_step": e2e_s * 1e3, "steps": e2e_steps},
+            "gpu_launches": int(launches),
+            "clocks": clk,
+        }
+        print(json.dumps(line))
+    h.h2tap_close(eng)
+    if world > 1:
+        dist.destroy_process_group()
+    return 0
+
+
+if __name__ == "__main__":
+    sys.exit(main())

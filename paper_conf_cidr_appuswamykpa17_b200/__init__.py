@@ -1,0 +1,312 @@
+"""B200-native OLAP hot path of an H2TAP engine (Appuswamy et al., CIDR 2017).
+
+Thin Python binding of the C ABI in ``include/h2tap.h`` (``libh2tap.so``, built in-tree by
+``_build.py`` for sm_100a). Every function here only marshals arguments: the snapshot store,
+the query kernels, the NCCL merge and the finalisation all run in the CUDA library. There is
+no CPU fallback — importing this package fails loudly when the library is missing.
+
+Names mirror the ABI: ``h2tap_open``, ``h2tap_load_snapshot``, ``h2tap_sync``,
+``h2tap_run_query``, ``h2tap_free``, ``h2tap_close``, ``h2tap_last_error``,
+``h2tap_nccl_unique_id``, ``h2tap_compute_stream``, ``h2tap_c_last_name``.
+"""
+from __future__ import annotations
+
+import ctypes as C
+import os
+
+import numpy as np
+
+_PKG = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_PKG, "libh2tap.so")
+
+if not os.path.exists(LIB_PATH):
+    raise ImportError(
+        f"{LIB_PATH} is missing: build it with `python -m paper_conf_cidr_appuswamykpa17_b200._build` "
+        "(or __graft_entry__.build()). There is no CPU fallback.")
+
+_lib = C.CDLL(LIB_PATH)
+
+# ------------------------------------------------------------------ ABI types --
+H2TAP_OK, H2TAP_EINVAL, H2TAP_ESTALE, H2TAP_ENOMEM = 0, -1, -2, -3
+H2TAP_ECUDA, H2TAP_ENCCL, H2TAP_EPLAN, H2TAP_EDUPKEY, H2TAP_ESHAPE = -4, -5, -6, -7, -8
+STATUS_NAMES = {0: "OK", -1: "EINVAL", -2: "ESTALE", -3: "ENOMEM", -4: "ECUDA", -5: "ENCCL",
+                -6: "EPLAN", -7: "EDUPKEY", -8: "ESHAPE", -9: "EOVERFLOW"}
+H2TAP_I32, H2TAP_I64, H2TAP_F64 = 1, 2, 3
+H2TAP_T_ORDER_LINE, H2TAP_T_ORDERS, H2TAP_T_CUSTOMER, H2TAP_T_ITEM = 1, 2, 3, 4
+H2TAP_Q1, H2TAP_Q6, H2TAP_Q18 = 1, 6, 18
+H2TAP_FULL_RELOAD = 1
+H2TAP_LOAD_ASYNC = 1
+H2TAP_RESULT_DEVICE = 1
+H2TAP_QUERY_PROFILE = 2
+
+_DT = {H2TAP_I32: np.int32, H2TAP_I64: np.int64, H2TAP_F64: np.float64}
+
+# Column ids per table, in header order (h2tap.h), keyed by the generator's column names.
+SCHEMA = {
+    "order_line": (H2TAP_T_ORDER_LINE, [
+        ("ol_w_id", H2TAP_I32), ("ol_d_id", H2TAP_I32), ("ol_o_id", H2TAP_I32),
+        ("ol_number", H2TAP_I32), ("ol_i_id", H2TAP_I32), ("ol_supply_w_id", H2TAP_I32),
+        ("ol_delivery_d", H2TAP_I64), ("ol_quantity", H2TAP_I32), ("ol_amount", H2TAP_I64)]),
+    "orders": (H2TAP_T_ORDERS, [
+        ("o_w_id", H2TAP_I32), ("o_d_id", H2TAP_I32), ("o_id", H2TAP_I32), ("o_c_id", H2TAP_I32),
+        ("o_ol_cnt", H2TAP_I32), ("o_carrier_id", H2TAP_I32), ("o_all_local", H2TAP_I32),
+        ("o_entry_d", H2TAP_I64)]),
+    "customer": (H2TAP_T_CUSTOMER, [
+        ("c_w_id", H2TAP_I32), ("c_d_id", H2TAP_I32), ("c_id", H2TAP_I32), ("c_last", H2TAP_I32)]),
+    "item": (H2TAP_T_ITEM, [("i_id", H2TAP_I32), ("i_price", H2TAP_I64)]),
+}
+
+
+class h2tap_column(C.Structure):
+    _fields_ = [("column_id", C.c_uint32), ("type", C.c_uint32), ("host_data", C.c_void_p)]
+
+
+class h2tap_table(C.Structure):
+    _fields_ = [("table_id", C.c_uint32), ("ncols", C.c_uint32), ("cols", C.POINTER(h2tap_column)),
+                ("row_count", C.c_uint64), ("first_row", C.c_uint64), ("flags", C.c_uint32)]
+
+
+class h2tap_config(C.Structure):
+    _fields_ = [("device", C.c_int), ("rank", C.c_int), ("world", C.c_int),
+                ("nccl_unique_id", C.c_void_p)]
+
+
+class h2tap_result(C.Structure):
+    _fields_ = [("epoch", C.c_uint64), ("nrows", C.c_uint64), ("ncols", C.c_uint32),
+                ("on_device", C.c_uint32), ("names", C.POINTER(C.c_char_p)),
+                ("types", C.POINTER(C.c_uint32)), ("cols", C.POINTER(C.c_void_p)),
+                ("nulls", C.POINTER(C.POINTER(C.c_uint8))), ("rows_scanned", C.c_uint64),
+                ("device_ms", C.c_double), ("e2e_ms", C.c_double), ("nkernels", C.c_uint32),
+                ("kernel_names", C.POINTER(C.c_char_p)), ("kernel_ms", C.POINTER(C.c_double)),
+                ("kernel_launches", C.c_uint64)]
+
+
+_P = C.c_void_p
+_lib.h2tap_open.argtypes = [C.POINTER(h2tap_config), C.POINTER(_P)]
+_lib.h2tap_load_snapshot_ex.argtypes = [_P, C.POINTER(h2tap_table), C.c_uint32, C.c_uint64, C.c_uint32]
+_lib.h2tap_load_snapshot.argtypes = [_P, C.POINTER(h2tap_table), C.c_uint32, C.c_uint64]
+_lib.h2tap_sync.argtypes = [_P, C.POINTER(C.c_uint64)]
+_lib.h2tap_run_query_ex.argtypes = [_P, C.c_uint32, C.POINTER(C.c_int64), C.c_uint32, C.c_uint32,
+                                    C.POINTER(C.POINTER(h2tap_result))]
+_lib.h2tap_run_query.argtypes = [_P, C.c_uint32, C.POINTER(C.c_int64), C.c_uint32,
+                                 C.POINTER(C.POINTER(h2tap_result))]
+_lib.h2tap_free.argtypes = [C.POINTER(h2tap_result)]
+_lib.h2tap_free.restype = None
+_lib.h2tap_close.argtypes = [_P]
+_lib.h2tap_close.restype = None
+_lib.h2tap_last_error.restype = C.c_char_p
+_lib.h2tap_nccl_unique_id.argtypes = [_P]
+_lib.h2tap_compute_stream.argtypes = [_P, C.POINTER(_P)]
+_lib.h2tap_c_last_name.argtypes = [C.c_int32, C.c_char_p, C.c_size_t]
+for _f in ("h2tap_open", "h2tap_load_snapshot_ex", "h2tap_load_snapshot", "h2tap_sync",
+           "h2tap_run_query_ex", "h2tap_run_query", "h2tap_nccl_unique_id", "h2tap_compute_stream"):
+    getattr(_lib, _f).restype = C.c_int
+
+ABI_SYMBOLS = ["h2tap_open", "h2tap_load_snapshot", "h2tap_load_snapshot_ex", "h2tap_sync",
+               "h2tap_run_query", "h2tap_run_query_ex", "h2tap_free", "h2tap_close",
+               "h2tap_last_error", "h2tap_nccl_unique_id", "h2tap_compute_stream",
+               "h2tap_c_last_name"]
+
+
+class H2tapError(RuntimeError):
+    def __init__(self, status, msg):
+        super().__init__(f"H2TAP_{STATUS_NAMES.get(status, status)}: {msg}")
+        self.status = status
+
+
+def h2tap_last_error() -> str:
+    return (_lib.h2tap_last_error() or b"").decode()
+
+
+def _check(st):
+    if st != H2TAP_OK:
+        raise H2tapError(st, h2tap_last_error())
+
+
+# ------------------------------------------------------------------ wrappers --
+class Engine:
+    """Handle of one engine (one GPU rank). Use h2tap_close() or the context manager."""
+
+    def __init__(self, handle, device, rank, world):
+        self.handle, self.device, self.rank, self.world = handle, device, rank, world
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *exc):
+        h2tap_close(self)
+
+
+def h2tap_nccl_unique_id() -> bytes:
+    buf = C.create_string_buffer(128)
+    _check(_lib.h2tap_nccl_unique_id(C.cast(buf, _P)))
+    return buf.raw
+
+
+def h2tap_open(device: int = 0, rank: int = 0, world: int = 1, nccl_unique_id: bytes | None = None) -> Engine:
+    idbuf = C.create_string_buffer(nccl_unique_id, 128) if nccl_unique_id is not None else None
+    cfg = h2tap_config(device, rank, world, C.cast(idbuf, _P) if idbuf is not None else None)
+    h = _P()
+    _check(_lib.h2tap_open(C.byref(cfg), C.byref(h)))
+    return Engine(h, device, rank, world)
+
+
+def h2tap_close(engine: Engine) -> None:
+    if engine is not None and engine.handle:
+        _lib.h2tap_close(engine.handle)
+        engine.handle = None
+
+
+def _host_ptr(a, want_dtype, name):
+    """Host pointer of a contiguous numpy array or CPU torch tensor (pinned or not)."""
+    if hasattr(a, "data_ptr") and hasattr(a, "is_cuda"):
+        if a.is_cuda:
+            raise ValueError(f"{name}: column buffers are host memory (the snapshot is refreshed H2D)")
+        if not a.is_contiguous() or a.element_size() != np.dtype(want_dtype).itemsize:
+            raise ValueError(f"{name}: needs a contiguous {np.dtype(want_dtype).name} tensor")
+        return a.data_ptr(), a, a.numel()
+    arr = np.ascontiguousarray(a)
+    if arr.dtype != want_dtype:
+        raise ValueError(f"{name}: dtype {arr.dtype}, schema wants {np.dtype(want_dtype).name}")
+    return arr.ctypes.data, arr, arr.size
+
+
+def h2tap_load_snapshot(engine: Engine, tables: dict, epoch: int, *, flags: int = 0,
+                        full_reload=True, first_row: dict | None = None) -> None:
+    """Refresh the device snapshot to ``epoch``.
+
+    ``tables``: {table_name: {column_name: array}} with the generator's names. Each array holds
+    rows [first_row, row_count) of its column. ``full_reload`` (bool, or a set of table names)
+    replaces those tables; other tables are appended to (``first_row[table]`` = rows already
+    loaded). ``flags``: H2TAP_LOAD_ASYNC to return before the epoch is published.
+    """
+    first_row = first_row or {}
+    keep, tabs, colarrs = [], [], []
+    for tname, cols in tables.items():
+        tid, schema = SCHEMA[tname]
+        ids = {n: (i, t) for i, (n, t) in enumerate(schema)}
+        carr = (h2tap_column * len(cols))()
+        nrows = None
+        for k, (cname, a) in enumerate(cols.items()):
+            cid, ty = ids[cname]
+            ptr, obj, n = _host_ptr(a, _DT[ty], f"{tname}.{cname}")
+            keep.append(obj)
+            if nrows is None:
+                nrows = n
+            elif n != nrows:
+                raise ValueError(f"{tname}: columns have different lengths ({n} vs {nrows})")
+            carr[k] = h2tap_column(cid, ty, ptr)
+        full = full_reload if isinstance(full_reload, bool) else tname in full_reload
+        fr = 0 if full else int(first_row.get(tname, 0))
+        colarrs.append(carr)
+        tabs.append(h2tap_table(tid, len(cols), carr, fr + (nrows or 0), fr,
+                                H2TAP_FULL_RELOAD if full else 0))
+    tarr = (h2tap_table * len(tabs))(*tabs)
+    _check(_lib.h2tap_load_snapshot_ex(engine.handle, tarr, len(tabs), epoch, flags))
+    del keep, colarrs
+
+
+def h2tap_sync(engine: Engine) -> int:
+    ep = C.c_uint64()
+    _check(_lib.h2tap_sync(engine.handle, C.byref(ep)))
+    return ep.value
+
+
+class _DevArray:
+    """__cuda_array_interface__ view of a device result column (for torch.as_tensor)."""
+
+    def __init__(self, ptr, n, dtype):
+        self.__cuda_array_interface__ = {"shape": (n,), "typestr": np.dtype(dtype).str,
+                                         "data": (ptr or 0, False), "version": 3, "strides": None}
+
+
+class Result:
+    """A query result. ``columns``: name -> numpy array (zero-copy view of library-owned pinned
+    memory, valid until h2tap_free) or, for device results, a __cuda_array_interface__ object.
+    ``nulls``: name -> uint8 array, only for columns that can hold NULL."""
+
+    def __init__(self, ptr):
+        self._ptr = ptr
+        r = ptr.contents
+        self.epoch, self.nrows, self.on_device = r.epoch, r.nrows, bool(r.on_device)
+        self.rows_scanned, self.device_ms, self.e2e_ms = r.rows_scanned, r.device_ms, r.e2e_ms
+        self.columns, self.nulls = {}, {}
+        for i in range(r.ncols):
+            name = r.names[i].decode()
+            dt = _DT[r.types[i]]
+            p = r.cols[i]
+            if self.on_device:
+                self.columns[name] = _DevArray(p, self.nrows, dt)
+            elif self.nrows:
+                self.columns[name] = np.ctypeslib.as_array(C.cast(p, C.POINTER(np.ctypeslib.as_ctypes_type(dt))), (self.nrows,))
+            else:
+                self.columns[name] = np.zeros(0, dt)
+            if bool(r.nulls[i]):
+                self.nulls[name] = np.ctypeslib.as_array(r.nulls[i], (self.nrows,)).copy()
+        self.kernel_launches = r.kernel_launches
+        self.kernels = [(r.kernel_names[i].decode(), r.kernel_ms[i]) for i in range(r.nkernels)]
+
+    def to_numpy(self) -> dict:
+        """Copy every column to a fresh host numpy array (device results via torch)."""
+        if not self.on_device:
+            return {k: np.array(v, copy=True) for k, v in self.columns.items()}
+        import torch
+        return {k: torch.as_tensor(v, device="cuda").cpu().numpy() if self.nrows else
+                np.zeros(0, np.dtype(v.__cuda_array_interface__["typestr"]))
+                for k, v in self.columns.items()}
+
+    def free(self):
+        h2tap_free(self)
+
+
+def h2tap_run_query(engine: Engine, plan: int, params=None, *, flags: int = 0) -> Result:
+    """Run plan H2TAP_Q1 / H2TAP_Q6 / H2TAP_Q18 (params: list of int64, None = CH defaults)."""
+    params = list(params or [])
+    parr = (C.c_int64 * max(1, len(params)))(*params)
+    out = C.POINTER(h2tap_result)()
+    _check(_lib.h2tap_run_query_ex(engine.handle, plan, parr, len(params), flags, C.byref(out)))
+    return Result(out)
+
+
+def h2tap_free(result: Result) -> None:
+    if result is not None and result._ptr:
+        _lib.h2tap_free(result._ptr)
+        result._ptr = None
+        result.columns = {}
+
+
+def h2tap_compute_stream(engine: Engine) -> int:
+    s = _P()
+    _check(_lib.h2tap_compute_stream(engine.handle, C.byref(s)))
+    return s.value or 0
+
+
+def h2tap_c_last_name(code: int) -> str:
+    buf = C.create_string_buffer(32)
+    n = _lib.h2tap_c_last_name(code, buf, 32)
+    if n < 0:
+        raise ValueError(f"c_last code {code} outside 0..999")
+    return buf.value.decode()
+
+
+def plan_columns():
+    """Columns each plan reads (what h2tap_load_snapshot must have provided)."""
+    return {
+        H2TAP_Q6: {"order_line": ["ol_delivery_d", "ol_quantity", "ol_amount"]},
+        H2TAP_Q1: {"order_line": ["ol_number", "ol_delivery_d", "ol_quantity", "ol_amount"]},
+        H2TAP_Q18: {"order_line": ["ol_w_id", "ol_d_id", "ol_o_id", "ol_amount"],
+                    "orders": ["o_w_id", "o_d_id", "o_id", "o_c_id", "o_ol_cnt", "o_entry_d"],
+                    "customer": ["c_w_id", "c_d_id", "c_id", "c_last"]},
+    }
+
+
+def hot_path_tables(tables: dict) -> dict:
+    """The subset of generated columns the hot path's plans read (union over Q1/Q6/Q18)."""
+    want = {}
+    for spec in plan_columns().values():
+        for t, cols in spec.items():
+            want.setdefault(t, [])
+            for c in cols:
+                if c not in want[t]:
+                    want[t].append(c)
+    return {t: {c: tables[t][c] for c in cols} for t, cols in want.items()}

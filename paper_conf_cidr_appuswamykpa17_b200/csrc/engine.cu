@@ -1,0 +1,1030 @@
+// engine.cu — the C ABI (include/h2tap.h): snapshot store in HBM with epoch publish (a1),
+// plan executors for CH Q1 / Q6 / Q18 (a2-a6, a8), NCCL merge across ranks (a7).
+//
+// Paper anchors:
+//  - snapshot = shallow copy of the top-level container + epoch++ (L562-567); here a View is
+//    an immutable {epoch, row count and device pointer per column}; appended rows go past every
+//    published count, so earlier views stay valid (the append-only subset of copy-on-write,
+//    L573-586) and views pin their buffers by reference count (the paper's epoch GC, L583-586).
+//  - several queries may share one snapshot, or take one each (L555-559): run_query reads the
+//    latest published view at entry; load_snapshot publishes a new one.
+//  - "the runtime identifies the columns that are necessary for executing the OLAP query and
+//    invokes the GPU kernel, passing in pointers" (L568-570): plans read only their columns.
+#include <algorithm>
+#include <atomic>
+#include <chrono>
+#include <cstdarg>
+#include <cstdio>
+#include <cstring>
+#include <deque>
+#include <map>
+#include <memory>
+#include <mutex>
+#include <string>
+#include <vector>
+
+#include <cuda_runtime.h>
+#include <nccl.h>
+
+#include "../../include/h2tap.h"
+#include "kernels.cuh"
+
+namespace h2tap {
+static std::atomic<uint64_t> g_launches{0};
+void count_launches(int n) { g_launches.fetch_add((uint64_t)n, std::memory_order_relaxed); }
+uint64_t launches_total() { return g_launches.load(std::memory_order_relaxed); }
+}  // namespace h2tap
+
+using namespace h2tap;
+
+// ============================================================== errors ===
+namespace {
+thread_local std::string g_err;
+
+h2tap_status fail(h2tap_status st, const char *fmt, ...) {
+    char buf[512];
+    va_list ap;
+    va_start(ap, fmt);
+    vsnprintf(buf, sizeof buf, fmt, ap);
+    va_end(ap);
+    g_err = buf;
+    return st;
+}
+
+struct Fail {  // thrown internally, converted to a status at the ABI boundary
+    h2tap_status st;
+};
+[[noreturn]] void raise(h2tap_status st, const char *fmt, ...) {
+    char buf[512];
+    va_list ap;
+    va_start(ap, fmt);
+    vsnprintf(buf, sizeof buf, fmt, ap);
+    va_end(ap);
+    g_err = buf;
+    throw Fail{st};
+}
+#define CK(call)                                                                           \
+    do {                                                                                   \
+        cudaError_t e_ = (call);                                                           \
+        if (e_ != cudaSuccess)                                                             \
+            raise(e_ == cudaErrorMemoryAllocation ? H2TAP_ENOMEM : H2TAP_ECUDA, "%s: %s (%s:%d)", \
+                  #call, cudaGetErrorString(e_), __FILE__, __LINE__);                      \
+    } while (0)
+#define NK(call)                                                                           \
+    do {                                                                                   \
+        ncclResult_t r_ = (call);                                                          \
+        if (r_ != ncclSuccess)                                                             \
+            raise(H2TAP_ENCCL, "%s: %s (%s:%d)", #call, ncclGetErrorString(r_), __FILE__,  \
+                  __LINE__);                                                               \
+    } while (0)
+
+// ============================================================== schema ===
+constexpr int kTables = 5;  // index = table id (1..4)
+constexpr int kMaxCols = 9;
+const int kNcols[kTables] = {0, 9, 8, 4, 2};
+const uint32_t kTypes[kTables][kMaxCols] = {
+    {},
+    {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64},
+    {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64},
+    {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32},
+    {H2TAP_I32, H2TAP_I64}};
+inline size_t type_size(uint32_t t) { return t == H2TAP_I32 ? 4 : 8; }
+constexpr uint64_t kPadRows = 64;  // over-allocation so 128-bit loads of the last tile stay in bounds
+
+// ============================================================ memory ===
+struct DevBuf {  // one device allocation; freed when the last View referencing it dies
+    void *ptr = nullptr;
+    size_t bytes = 0;
+    int device = 0;
+    ~DevBuf() {
+        if (ptr) {
+            int cur;
+            cudaGetDevice(&cur);
+            cudaSetDevice(device);
+            cudaFree(ptr);
+            cudaSetDevice(cur);
+        }
+    }
+};
+using DevBufP = std::shared_ptr<DevBuf>;
+
+DevBufP dev_alloc(size_t bytes, int device) {
+    auto b = std::make_shared<DevBuf>();
+    b->device = device;
+    b->bytes = bytes;
+    CK(cudaMalloc(&b->ptr, bytes ? bytes : 16));
+    return b;
+}
+
+// Pool of pinned host blocks (result columns) and of device blocks (device-resident results).
+struct BlockPool {
+    bool pinned;  // true: cudaMallocHost, false: cudaMalloc
+    int device;
+    std::mutex mu;
+    std::multimap<size_t, void *> free_blocks;
+    BlockPool(bool p, int d) : pinned(p), device(d) {}
+    ~BlockPool() {
+        int cur;
+        cudaGetDevice(&cur);
+        cudaSetDevice(device);
+        for (auto &kv : free_blocks) pinned ? cudaFreeHost(kv.second) : cudaFree(kv.second);
+        cudaSetDevice(cur);
+    }
+    static size_t size_class(size_t b) {
+        size_t s = 4096;
+        while (s < b) s <<= 1;
+        return s;
+    }
+    std::pair<void *, size_t> get(size_t bytes) {
+        const size_t sc = size_class(bytes);
+        {
+            std::lock_guard<std::mutex> g(mu);
+            auto it = free_blocks.find(sc);
+            if (it != free_blocks.end()) {
+                void *p = it->second;
+                free_blocks.erase(it);
+                return {p, sc};
+            }
+        }
+        void *p = nullptr;
+        if (pinned) CK(cudaMallocHost(&p, sc));
+        else CK(cudaMalloc(&p, sc));
+        return {p, sc};
+    }
+    void put(void *p, size_t sc) {
+        std::lock_guard<std::mutex> g(mu);
+        free_blocks.emplace(sc, p);
+    }
+};
+
+// ============================================================ results ===
+struct ResultImpl : h2tap_result {
+    std::vector<std::string> name_store;
+    std::vector<const char *> name_ptrs;
+    std::vector<uint32_t> type_store;
+    std::vector<const void *> col_ptrs;
+    std::vector<std::vector<uint8_t>> null_store;
+    std::vector<const uint8_t *> null_ptrs;
+    std::vector<std::string> kname_store;
+    std::vector<const char *> kname_ptrs;
+    std::vector<double> kms;
+    std::vector<std::pair<void *, size_t>> blocks;
+    std::shared_ptr<BlockPool> pool;
+    ~ResultImpl() {
+        if (pool)
+            for (auto &b : blocks) pool->put(b.first, b.second);
+    }
+    void finish() {
+        name_ptrs.clear();
+        for (auto &s : name_store) name_ptrs.push_back(s.c_str());
+        null_ptrs.clear();
+        for (auto &v : null_store) null_ptrs.push_back(v.empty() ? nullptr : v.data());
+        kname_ptrs.clear();
+        for (auto &s : kname_store) kname_ptrs.push_back(s.c_str());
+        names = name_ptrs.data();
+        types = type_store.data();
+        cols = col_ptrs.data();
+        nulls = null_ptrs.data();
+        ncols = (uint32_t)name_store.size();
+        nkernels = (uint32_t)kname_store.size();
+        kernel_names = kname_ptrs.data();
+        kernel_ms = kms.data();
+    }
+};
+
+// =========================================================== snapshot ===
+struct View {  // immutable snapshot at one epoch (the paper's shallow-copied top container)
+    uint64_t epoch = 0;
+    uint64_t n[kTables] = {};
+    void *col[kTables][kMaxCols] = {};
+    DevBufP keep[kTables][kMaxCols];
+};
+using ViewP = std::shared_ptr<const View>;
+
+struct ColState {
+    DevBufP cur, spare;
+    uint64_t cap_rows = 0;
+};
+struct TableState {
+    bool present = false;
+    uint32_t colmask = 0;   // which column ids this table carries (fixed at first load)
+    uint64_t loaded = 0;    // rows copied or in flight
+    ColState col[kMaxCols];
+};
+
+struct Pending {
+    uint64_t epoch;
+    ViewP view;
+    cudaEvent_t done;
+};
+
+struct Staging {  // pinned ring for pageable host buffers
+    static constexpr size_t kChunk = 32u << 20;
+    static constexpr int kSlots = 3;
+    void *buf[kSlots] = {};
+    cudaEvent_t ev[kSlots] = {};
+    int next = 0;
+};
+
+// ============================================================ scratch ===
+struct Arena {  // grow-only named device buffers, owned by the engine
+    std::map<std::string, DevBufP> bufs;
+    int device = 0;
+    void *get(const std::string &name, size_t bytes, bool zero = false, cudaStream_t st = nullptr) {
+        auto &b = bufs[name];
+        if (!b || b->bytes < bytes) {
+            if (b) CK(cudaDeviceSynchronize());  // old buffer may still be in use on a stream
+            b.reset();
+            b = dev_alloc(bytes, device);
+            if (zero) CK(cudaMemsetAsync(b->ptr, 0, b->bytes, st));
+        }
+        return b->ptr;
+    }
+};
+
+struct Prof {  // per-kernel CUDA events on the compute stream
+    bool on = false;
+    cudaStream_t st = nullptr;
+    std::vector<std::pair<std::string, std::pair<cudaEvent_t, cudaEvent_t>>> marks;
+    std::vector<cudaEvent_t> pool;
+    size_t used = 0;
+    cudaEvent_t ev() {
+        if (used == pool.size()) {
+            cudaEvent_t e;
+            CK(cudaEventCreate(&e));
+            pool.push_back(e);
+        }
+        return pool[used++];
+    }
+    template <class F> void run(const char *name, F &&f) {
+        if (!on) { f(); return; }
+        cudaEvent_t a = ev(), b = ev();
+        CK(cudaEventRecord(a, st));
+        f();
+        CK(cudaEventRecord(b, st));
+        marks.push_back({name, {a, b}});
+    }
+    void reset(bool enable, cudaStream_t s) { on = enable; st = s; marks.clear(); used = 0; }
+};
+
+}  // namespace
+
+// ============================================================= engine ===
+struct h2tap_engine {
+    int device = 0, rank = 0, world = 1, num_sms = 148;
+    ncclComm_t comm = nullptr;
+    cudaStream_t compute = nullptr, copy = nullptr;
+    cudaEvent_t q_begin = nullptr, q_end = nullptr;
+
+    std::mutex load_mu, query_mu, view_mu, pend_mu;
+    TableState tables[kTables];
+    ViewP published;
+    ViewP accepted;               // latest accepted (published or pending) view
+    std::atomic<uint64_t> last_epoch{0};
+    bool any_epoch = false;
+    std::deque<Pending> pending;
+    Staging staging;
+
+    Arena arena;
+    Prof prof;
+    std::shared_ptr<BlockPool> host_pool, dev_pool;
+    long long *small_host = nullptr;  // pinned scratch for tiny D2H reads
+};
+
+namespace {
+
+void publish_ready(h2tap_engine *e, bool wait) {
+    std::lock_guard<std::mutex> g(e->pend_mu);
+    while (!e->pending.empty()) {
+        Pending &p = e->pending.front();
+        if (wait) CK(cudaEventSynchronize(p.done));
+        else {
+            cudaError_t q = cudaEventQuery(p.done);
+            if (q == cudaErrorNotReady) break;
+            if (q != cudaSuccess) CK(q);
+        }
+        {
+            std::lock_guard<std::mutex> gv(e->view_mu);
+            e->published = p.view;
+        }
+        cudaEventDestroy(p.done);
+        e->pending.pop_front();
+    }
+}
+
+bool host_is_pinned(const void *p) {
+    cudaPointerAttributes a;
+    if (cudaPointerGetAttributes(&a, p) != cudaSuccess) {
+        cudaGetLastError();
+        return false;
+    }
+    return a.type == cudaMemoryTypeHost;
+}
+
+// Copy `bytes` from host `src` to device `dst` on the copy stream. Pinned sources are DMA'd
+// directly (returns true: the caller must wait before returning); pageable ones go through the
+// pinned staging ring (the engine owns those bytes once memcpy'd, so no wait is needed).
+bool h2d(h2tap_engine *e, void *dst, const void *src, size_t bytes) {
+    if (!bytes) return false;
+    if (host_is_pinned(src)) {
+        CK(cudaMemcpyAsync(dst, src, bytes, cudaMemcpyHostToDevice, e->copy));
+        return true;
+    }
+    Staging &S = e->staging;
+    for (size_t off = 0; off < bytes; off += Staging::kChunk) {
+        const size_t len = std::min(Staging::kChunk, bytes - off);
+        const int k = S.next;
+        S.next = (S.next + 1) % Staging::kSlots;
+        if (!S.buf[k]) {
+            CK(cudaMallocHost(&S.buf[k], Staging::kChunk));
+            CK(cudaEventCreateWithFlags(&S.ev[k], cudaEventDisableTiming));
+        } else {
+            CK(cudaEventSynchronize(S.ev[k]));  // previous DMA out of this slot has drained
+        }
+        std::memcpy(S.buf[k], static_cast<const char *>(src) + off, len);
+        CK(cudaMemcpyAsync(static_cast<char *>(dst) + off, S.buf[k], len, cudaMemcpyHostToDevice,
+                           e->copy));
+        CK(cudaEventRecord(S.ev[k], e->copy));
+    }
+    return false;
+}
+
+h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntables,
+                       uint64_t epoch, uint32_t flags) {
+    std::lock_guard<std::mutex> g(e->load_mu);
+    CK(cudaSetDevice(e->device));
+    publish_ready(e, false);
+    if (e->any_epoch && epoch <= e->last_epoch.load())
+        return fail(H2TAP_ESTALE, "epoch %llu is not greater than the last accepted epoch %llu",
+                    (unsigned long long)epoch, (unsigned long long)e->last_epoch.load());
+    if (ntables && !tables) return fail(H2TAP_EINVAL, "tables is NULL");
+    // ---- validate everything before touching state
+    bool seen[kTables] = {};
+    for (uint32_t i = 0; i < ntables; ++i) {
+        const h2tap_table &t = tables[i];
+        if (t.table_id < 1 || t.table_id > 4) return fail(H2TAP_EINVAL, "unknown table id %u", t.table_id);
+        if (seen[t.table_id]) return fail(H2TAP_EINVAL, "table %u listed twice", t.table_id);
+        seen[t.table_id] = true;
+        if (t.ncols == 0 || !t.cols) return fail(H2TAP_EINVAL, "table %u has no columns", t.table_id);
+        if (t.row_count < t.first_row) return fail(H2TAP_EINVAL, "table %u: row_count < first_row", t.table_id);
+        if (t.row_count >= (1ull << 31)) return fail(H2TAP_EINVAL, "table %u: more than 2^31-1 rows", t.table_id);
+        uint32_t mask = 0;
+        for (uint32_t c = 0; c < t.ncols; ++c) {
+            const h2tap_column &col = t.cols[c];
+            if (col.column_id >= (uint32_t)kNcols[t.table_id])
+                return fail(H2TAP_EINVAL, "table %u: unknown column id %u", t.table_id, col.column_id);
+            if (col.type != kTypes[t.table_id][col.column_id])
+                return fail(H2TAP_EINVAL, "table %u column %u: type %u, schema type %u", t.table_id,
+                            col.column_id, col.type, kTypes[t.table_id][col.column_id]);
+            if (mask & (1u << col.column_id))
+                return fail(H2TAP_EINVAL, "table %u: column %u listed twice", t.table_id, col.column_id);
+            if (!col.host_data && t.row_count > t.first_row)
+                return fail(H2TAP_EINVAL, "table %u column %u: host_data is NULL", t.table_id, col.column_id);
+            mask |= 1u << col.column_id;
+        }
+        const TableState &ts = e->tables[t.table_id];
+        if (t.flags & H2TAP_FULL_RELOAD) {
+            if (t.first_row != 0) return fail(H2TAP_EINVAL, "table %u: full reload must start at row 0", t.table_id);
+        } else {
+            if (ts.present && mask != ts.colmask)
+                return fail(H2TAP_ESHAPE, "table %u: append column set differs from the loaded set", t.table_id);
+            if (t.first_row != ts.loaded)
+                return fail(H2TAP_ESHAPE, "table %u: append starts at row %llu but %llu rows are loaded",
+                            t.table_id, (unsigned long long)t.first_row, (unsigned long long)ts.loaded);
+        }
+    }
+    // ---- copy and build the new view
+    auto v = std::make_shared<View>();
+    if (e->accepted) *v = *e->accepted;
+    v->epoch = epoch;
+    bool must_wait = false;
+    for (uint32_t i = 0; i < ntables; ++i) {
+        const h2tap_table &t = tables[i];
+        TableState &ts = e->tables[t.table_id];
+        const bool full = t.flags & H2TAP_FULL_RELOAD;
+        if (full) {  // a full reload may change the column set
+            uint32_t mask = 0;
+            for (uint32_t c = 0; c < t.ncols; ++c) mask |= 1u << t.cols[c].column_id;
+            for (int c = 0; c < kNcols[t.table_id]; ++c)
+                if (!(mask & (1u << c))) {
+                    v->col[t.table_id][c] = nullptr;
+                    v->keep[t.table_id][c].reset();
+                    ts.col[c] = ColState{};
+                }
+            ts.colmask = mask;
+        }
+        for (uint32_t c = 0; c < t.ncols; ++c) {
+            const h2tap_column &col = t.cols[c];
+            ColState &cs = ts.col[col.column_id];
+            const size_t es = type_size(col.type);
+            const uint64_t need = t.row_count + kPadRows;
+            if (full) {
+                // never overwrite a buffer a live view may read: reuse the spare only when no
+                // view references it any more, else allocate
+                DevBufP target;
+                if (cs.spare && cs.spare.use_count() == 1 && cs.spare->bytes >= need * es) target = cs.spare;
+                else target = dev_alloc(need * es + need * es / 8, e->device);
+                cs.spare = cs.cur;
+                cs.cur = target;
+                cs.cap_rows = target->bytes / es;
+            } else if (!cs.cur || need > cs.cap_rows) {
+                // grow: new buffer, device-to-device copy of the visible prefix; the old buffer
+                // stays alive for views that still reference it
+                const uint64_t cap = std::max<uint64_t>(need, (cs.cap_rows * 3) / 2);
+                DevBufP nb = dev_alloc(cap * es, e->device);
+                if (cs.cur && t.first_row)
+                    CK(cudaMemcpyAsync(nb->ptr, cs.cur->ptr, t.first_row * es, cudaMemcpyDeviceToDevice, e->copy));
+                cs.spare.reset();
+                cs.cur = nb;
+                cs.cap_rows = cap;
+            }
+            must_wait |= h2d(e, static_cast<char *>(cs.cur->ptr) + t.first_row * es, col.host_data,
+                             (t.row_count - t.first_row) * es);
+            v->col[t.table_id][col.column_id] = cs.cur->ptr;
+            v->keep[t.table_id][col.column_id] = cs.cur;
+        }
+        ts.present = true;
+        if (!full) {
+            uint32_t mask = 0;
+            for (uint32_t c = 0; c < t.ncols; ++c) mask |= 1u << t.cols[c].column_id;
+            ts.colmask = mask;
+        }
+        ts.loaded = t.row_count;
+        v->n[t.table_id] = t.row_count;
+    }
+    cudaEvent_t done;
+    CK(cudaEventCreateWithFlags(&done, cudaEventDisableTiming));
+    CK(cudaEventRecord(done, e->copy));
+    e->accepted = v;
+    e->last_epoch = epoch;
+    e->any_epoch = true;
+    {
+        std::lock_guard<std::mutex> gp(e->pend_mu);
+        e->pending.push_back(Pending{epoch, v, done});
+    }
+    if (must_wait || !(flags & H2TAP_LOAD_ASYNC)) publish_ready(e, true);
+    return H2TAP_OK;
+}
+
+// ------------------------------------------------------------ plans --
+struct Col { const void *p; };
+template <class T> const T *colp(const View &v, int t, int c) {
+    return static_cast<const T *>(v.col[t][c]);
+}
+
+void need_cols(const View &v, int t, std::initializer_list<int> cs, const char *plan) {
+    for (int c : cs)
+        if (!v.col[t][c] && v.n[t])
+            raise(H2TAP_EPLAN, "%s needs column %d of table %d, which was never loaded", plan, c, t);
+}
+
+ResultImpl *new_result(h2tap_engine *e, const View &v, bool dev) {
+    auto *r = new ResultImpl();
+    std::memset(static_cast<h2tap_result *>(r), 0, sizeof(h2tap_result));
+    r->epoch = v.epoch;
+    r->rows_scanned = v.n[H2TAP_T_ORDER_LINE];
+    r->on_device = dev ? 1 : 0;
+    r->pool = dev ? e->dev_pool : e->host_pool;
+    return r;
+}
+
+// Allocate result column storage (pinned host or device) of `bytes`.
+void *result_block(ResultImpl *r, size_t bytes) {
+    auto b = r->pool->get(bytes ? bytes : 8);
+    r->blocks.push_back(b);
+    return b.first;
+}
+
+void add_col(ResultImpl *r, const char *name, uint32_t type, const void *p) {
+    r->name_store.emplace_back(name);
+    r->type_store.push_back(type);
+    r->col_ptrs.push_back(p);
+    r->null_store.emplace_back();
+}
+
+void sync_compute(h2tap_engine *e) { CK(cudaStreamSynchronize(e->compute)); }
+
+// ---- Q6 (a2 + a7)
+void run_q6(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
+    const int T = H2TAP_T_ORDER_LINE;
+    need_cols(v, T, {H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}, "Q6");
+    Q6Scratch s;
+    const int mb = q6_max_blocks(e->num_sms);
+    s.block_part = static_cast<long long *>(e->arena.get("q6.part", sizeof(long long) * 2 * mb));
+    s.done_counter = static_cast<unsigned int *>(e->arena.get("q6.counter", 64, true, e->compute));
+    s.out = static_cast<long long *>(e->arena.get("q6.out", 64));
+    e->prof.run("q6_scan_filter_sum", [&] {
+        launch_q6(colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D), colp<int32_t>(v, T, H2TAP_OL_QUANTITY),
+                  colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T], p[0], p[1], p[2], p[3], s,
+                  e->num_sms, e->compute);
+        CK(cudaGetLastError());
+    });
+    if (e->world > 1)
+        e->prof.run("q6_allreduce", [&] {
+            NK(ncclAllReduce(s.out, s.out, 2, ncclInt64, ncclSum, e->comm, e->compute));
+        });
+    CK(cudaMemcpyAsync(e->small_host, s.out, 16, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaEventRecord(e->q_end, e->compute));
+    sync_compute(e);
+    const long long rev = e->small_host[0], cnt = e->small_host[1];
+    r->nrows = 1;
+    auto *blk = static_cast<long long *>(result_block(r, 16));
+    if (r->on_device) CK(cudaMemcpy(blk, e->small_host, 16, cudaMemcpyHostToDevice));
+    else { blk[0] = rev; blk[1] = cnt; }
+    add_col(r, "revenue", H2TAP_I64, blk);
+    r->null_store.back().assign(1, cnt == 0 ? 1 : 0);  // SUM over no rows IS NULL (R8)
+    add_col(r, "count_rows", H2TAP_I64, blk + 1);
+}
+
+// ---- Q1 (a3 + a7 + a8)
+void run_q1(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
+    const int T = H2TAP_T_ORDER_LINE;
+    need_cols(v, T, {H2TAP_OL_NUMBER, H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}, "Q1");
+    Q1Scratch s;
+    const size_t maxg = kQ1GlobalSlots + kQ1Dense;
+    bool fresh = !e->arena.bufs.count("q1.gtag");
+    s.dense = static_cast<unsigned long long *>(e->arena.get("q1.dense", 8 * kQ1Dense * 3));
+    s.gtag = static_cast<unsigned long long *>(e->arena.get("q1.gtag", 8ull * kQ1GlobalSlots));
+    s.gacc = static_cast<unsigned long long *>(e->arena.get("q1.gacc", 24ull * kQ1GlobalSlots));
+    s.flags = static_cast<unsigned int *>(e->arena.get("q1.flags", 64));
+    s.groups = static_cast<Q1Group *>(e->arena.get("q1.groups", sizeof(Q1Group) * maxg));
+    s.ngroups = static_cast<unsigned long long *>(e->arena.get("q1.ngroups", 64));
+    s.o_key = static_cast<int32_t *>(e->arena.get("q1.okey", 4 * maxg));
+    s.o_qty = static_cast<long long *>(e->arena.get("q1.oqty", 8 * maxg));
+    s.o_amt = static_cast<long long *>(e->arena.get("q1.oamt", 8 * maxg));
+    s.o_cnt = static_cast<long long *>(e->arena.get("q1.ocnt", 8 * maxg));
+    s.o_avg_qty = static_cast<double *>(e->arena.get("q1.oavgq", 8 * maxg));
+    s.o_avg_amt = static_cast<double *>(e->arena.get("q1.oavga", 8 * maxg));
+    if (fresh) launch_q1_reset(s, e->compute);  // tables self-clean afterwards (q1_compact)
+    e->prof.run("q1_scan_filter_groupby", [&] {
+        launch_q1(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
+                  colp<int32_t>(v, T, H2TAP_OL_QUANTITY), colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T],
+                  p[0], s, e->num_sms, e->compute);
+        CK(cudaGetLastError());
+    });
+    e->prof.run("q1_compact", [&] { launch_q1_compact(s, e->compute); });
+    CK(cudaMemcpyAsync(e->small_host, s.ngroups, 8, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaMemcpyAsync(e->small_host + 1, s.flags, 4, cudaMemcpyDeviceToHost, e->compute));
+    sync_compute(e);
+    uint64_t ng = (uint64_t)e->small_host[0];
+    if (e->small_host[1] & 1) {
+        CK(cudaMemsetAsync(s.flags, 0, 4, e->compute));
+        raise(H2TAP_ENOMEM, "Q1: more than %d distinct ol_number groups", kQ1GlobalSlots);
+    }
+    if (e->world > 1) {  // a7: gather every rank's groups, fold into one table, re-compact
+        auto *cnt_dev = static_cast<unsigned long long *>(e->arena.get("q1.allcnt", 8ull * e->world));
+        e->prof.run("q1_allgather", [&] {
+            NK(ncclAllGather(s.ngroups, cnt_dev, 1, ncclUint64, e->comm, e->compute));
+        });
+        std::vector<unsigned long long> cnts(e->world);
+        CK(cudaMemcpyAsync(cnts.data(), cnt_dev, 8ull * e->world, cudaMemcpyDeviceToHost, e->compute));
+        sync_compute(e);
+        const uint64_t gcap = *std::max_element(cnts.begin(), cnts.end());
+        auto *all = static_cast<Q1Group *>(e->arena.get("q1.all", sizeof(Q1Group) * std::max<uint64_t>(gcap, 1) * e->world));
+        e->prof.run("q1_allgather_groups", [&] {
+            if (gcap)
+                NK(ncclAllGather(s.groups, all, gcap * sizeof(Q1Group), ncclUint8, e->comm, e->compute));
+        });
+        e->prof.run("q1_merge", [&] {
+            for (int k = 0; k < e->world; ++k)
+                if (cnts[k]) launch_q1_merge(all + (uint64_t)k * gcap, cnts[k], s, e->compute);
+            launch_q1_compact(s, e->compute);
+        });
+        CK(cudaMemcpyAsync(e->small_host, s.ngroups, 8, cudaMemcpyDeviceToHost, e->compute));
+        sync_compute(e);
+        ng = (uint64_t)e->small_host[0];
+    }
+    e->prof.run("q1_emit", [&] { launch_q1_emit(s, ng, e->compute); });
+    r->nrows = ng;
+    struct { const char *name; uint32_t type; const void *src; size_t es; } cols[] = {
+        {"ol_number", H2TAP_I32, s.o_key, 4}, {"sum_qty", H2TAP_I64, s.o_qty, 8},
+        {"sum_amount", H2TAP_I64, s.o_amt, 8}, {"avg_qty", H2TAP_F64, s.o_avg_qty, 8},
+        {"avg_amount", H2TAP_F64, s.o_avg_amt, 8}, {"count_order", H2TAP_I64, s.o_cnt, 8}};
+    for (auto &c : cols) {
+        void *dst = result_block(r, ng * c.es);
+        if (ng)
+            CK(cudaMemcpyAsync(dst, c.src, ng * c.es,
+                               r->on_device ? cudaMemcpyDeviceToDevice : cudaMemcpyDeviceToHost,
+                               e->compute));
+        add_col(r, c.name, c.type, dst);
+    }
+    CK(cudaEventRecord(e->q_end, e->compute));
+    sync_compute(e);
+}
+
+// ---- Q18 (a4 + a5 + a6 + a7 + a8)
+int bitwidth(unsigned long long x) { return x ? 64 - __builtin_clzll(x) : 0; }
+
+Q18Cols carve_cols(Arena &a, const char *prefix, uint64_t n) {
+    auto nm = [&](const char *c) { return std::string(prefix) + c; };
+    const uint64_t m = std::max<uint64_t>(n, 1);
+    Q18Cols c;
+    c.c_last = static_cast<int32_t *>(a.get(nm("c_last"), 4 * m));
+    c.c_id = static_cast<int32_t *>(a.get(nm("c_id"), 4 * m));
+    c.o_id = static_cast<int32_t *>(a.get(nm("o_id"), 4 * m));
+    c.o_ol_cnt = static_cast<int32_t *>(a.get(nm("o_ol_cnt"), 4 * m));
+    c.o_w_id = static_cast<int32_t *>(a.get(nm("o_w_id"), 4 * m));
+    c.o_d_id = static_cast<int32_t *>(a.get(nm("o_d_id"), 4 * m));
+    c.o_entry_d = static_cast<int64_t *>(a.get(nm("o_entry_d"), 8 * m));
+    c.amount_sum = static_cast<int64_t *>(a.get(nm("amount_sum"), 8 * m));
+    return c;
+}
+
+uint64_t pow2_at_least(uint64_t x) {
+    uint64_t c = 16;
+    while (c < x) c <<= 1;
+    return c;
+}
+
+void run_q18(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
+    const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
+    need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}, "Q18");
+    need_cols(v, O, {H2TAP_O_W_ID, H2TAP_O_D_ID, H2TAP_O_ID, H2TAP_O_C_ID, H2TAP_O_OL_CNT, H2TAP_O_ENTRY_D}, "Q18");
+    need_cols(v, C, {H2TAP_C_W_ID, H2TAP_C_D_ID, H2TAP_C_ID, H2TAP_C_LAST}, "Q18");
+    const uint64_t n_ol = v.n[OL], n_o = v.n[O], n_c = v.n[C];
+    Q18Scratch s;
+    s.cap_o = pow2_at_least(2 * n_o);
+    s.cap_c = pow2_at_least(2 * n_c);
+    s.ht_o = static_cast<HtSlot *>(e->arena.get("q18.ht_o", sizeof(HtSlot) * s.cap_o));
+    s.ht_c = static_cast<HtSlot *>(e->arena.get("q18.ht_c", sizeof(HtSlot) * s.cap_c));
+    s.acc = static_cast<Q18Acc *>(e->arena.get("q18.acc", sizeof(Q18Acc) * std::max<uint64_t>(n_o, 1)));
+    s.err = static_cast<unsigned int *>(e->arena.get("q18.err", 64));
+    s.nout = static_cast<unsigned long long *>(e->arena.get("q18.nout", 64));
+    s.stats = static_cast<Q18Stats *>(e->arena.get("q18.stats", sizeof(Q18Stats)));
+    s.un = carve_cols(e->arena, "q18.un.", n_o);
+
+    e->prof.run("q18_init", [&] { launch_q18_init(s, n_o, e->compute); });
+    e->prof.run("q18_build", [&] {
+        launch_q18_build(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
+                         colp<int32_t>(v, O, H2TAP_O_ID), n_o, colp<int32_t>(v, C, H2TAP_C_W_ID),
+                         colp<int32_t>(v, C, H2TAP_C_D_ID), colp<int32_t>(v, C, H2TAP_C_ID), n_c, s,
+                         e->num_sms, e->compute);
+    });
+    e->prof.run("q18_probe_groupjoin", [&] {
+        if (n_ol)
+            launch_q18_probe(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
+                             colp<int32_t>(v, OL, H2TAP_OL_O_ID), colp<int64_t>(v, OL, H2TAP_OL_AMOUNT),
+                             n_ol, s, e->num_sms, e->compute);
+    });
+    e->prof.run("q18_having_compact", [&] {
+        if (n_o)
+            launch_q18_having(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
+                              colp<int32_t>(v, O, H2TAP_O_ID), colp<int32_t>(v, O, H2TAP_O_C_ID),
+                              colp<int32_t>(v, O, H2TAP_O_OL_CNT), colp<int64_t>(v, O, H2TAP_O_ENTRY_D),
+                              n_o, colp<int32_t>(v, C, H2TAP_C_LAST), p[0], s, e->num_sms, e->compute);
+    });
+    CK(cudaGetLastError());
+    // small D2H: err, nout, stats
+    struct Small { unsigned long long nout; unsigned int err, pad; Q18Stats st; };
+    static_assert(sizeof(Small) <= 256, "small");
+    Small *sm = reinterpret_cast<Small *>(e->small_host);
+    CK(cudaMemcpyAsync(&sm->nout, s.nout, 8, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaMemcpyAsync(&sm->err, s.err, 4, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaMemcpyAsync(&sm->st, s.stats, sizeof(Q18Stats), cudaMemcpyDeviceToHost, e->compute));
+    sync_compute(e);
+    const unsigned int err = sm->err;
+    uint64_t nout = sm->nout;
+    Q18Stats st = sm->st;
+    int err_any = err ? 1 : 0;
+    if (e->world > 1) {  // every rank must learn whether any rank failed before the next collective
+        auto *flag = static_cast<int *>(e->arena.get("q18.errflag", 64));
+        CK(cudaMemcpyAsync(flag, &err_any, 4, cudaMemcpyHostToDevice, e->compute));
+        NK(ncclAllReduce(flag, flag, 1, ncclInt32, ncclMax, e->comm, e->compute));
+        CK(cudaMemcpyAsync(&err_any, flag, 4, cudaMemcpyDeviceToHost, e->compute));
+        sync_compute(e);
+    }
+    if (err & kErrDupOrders) raise(H2TAP_EDUPKEY, "Q18: duplicate orders primary key (w, d, o_id)");
+    if (err & kErrDupCustomer) raise(H2TAP_EDUPKEY, "Q18: duplicate customer primary key (w, d, c_id)");
+    if (err & kErrDomain) raise(H2TAP_EPLAN, "Q18: join key outside the supported domain");
+    if (err_any) raise(H2TAP_EPLAN, "Q18: failed on another rank");
+
+    Q18Cols src = s.un;
+    if (e->world > 1) {  // a7: groups are warehouse-local; gather result rows to rank 0
+        auto *cnt_dev = static_cast<unsigned long long *>(e->arena.get("q18.allcnt", 8ull * e->world));
+        NK(ncclAllGather(s.nout, cnt_dev, 1, ncclUint64, e->comm, e->compute));
+        std::vector<unsigned long long> cnts(e->world);
+        CK(cudaMemcpyAsync(cnts.data(), cnt_dev, 8ull * e->world, cudaMemcpyDeviceToHost, e->compute));
+        sync_compute(e);
+        uint64_t total = 0;
+        for (auto c : cnts) total += c;
+        if (e->rank == 0) src = carve_cols(e->arena, "q18.all.", total);
+        e->prof.run("q18_gather", [&] {
+            NK(ncclGroupStart());
+            uint64_t off = 0;
+            for (int k = 0; k < e->world; ++k) {
+                const uint64_t c = cnts[k];
+                if (!c) continue;
+                auto xfer = [&](void *dst_base, const void *src_base, size_t es) {
+                    if (e->rank == 0 && k == 0)
+                        CK(cudaMemcpyAsync(static_cast<char *>(dst_base) + off * es, src_base, c * es,
+                                           cudaMemcpyDeviceToDevice, e->compute));
+                    else if (e->rank == 0)
+                        NK(ncclRecv(static_cast<char *>(dst_base) + off * es, c * es, ncclUint8, k, e->comm, e->compute));
+                    else if (e->rank == k)
+                        NK(ncclSend(src_base, c * es, ncclUint8, 0, e->comm, e->compute));
+                };
+                xfer(src.c_last, s.un.c_last, 4); xfer(src.c_id, s.un.c_id, 4);
+                xfer(src.o_id, s.un.o_id, 4); xfer(src.o_ol_cnt, s.un.o_ol_cnt, 4);
+                xfer(src.o_w_id, s.un.o_w_id, 4); xfer(src.o_d_id, s.un.o_d_id, 4);
+                xfer(src.o_entry_d, s.un.o_entry_d, 8); xfer(src.amount_sum, s.un.amount_sum, 8);
+                off += c;
+            }
+            NK(ncclGroupEnd());
+        });
+        if (e->rank != 0) {
+            CK(cudaEventRecord(e->q_end, e->compute));
+            sync_compute(e);
+            r->nrows = 0;
+            const char *names[] = {"c_last", "c_id", "o_id", "o_entry_d", "o_ol_cnt", "amount_sum", "o_w_id", "o_d_id"};
+            const uint32_t types[] = {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I32};
+            for (int i = 0; i < 8; ++i) add_col(r, names[i], types[i], result_block(r, 8));
+            return;
+        }
+        nout = total;
+        // stats over the gathered rows
+        Q18Stats init;
+        init.amt_min = INT64_MAX; init.amt_max = INT64_MIN; init.ent_min = INT64_MAX; init.ent_max = INT64_MIN;
+        init.w_min = INT32_MAX; init.w_max = INT32_MIN; init.d_min = INT32_MAX; init.d_max = INT32_MIN;
+        init.o_min = INT32_MAX; init.o_max = INT32_MIN; init.pad0 = init.pad1 = 0;
+        sm->st = init;
+        CK(cudaMemcpyAsync(s.stats, &sm->st, sizeof(Q18Stats), cudaMemcpyHostToDevice, e->compute));
+        launch_q18_stats(src, nout, s.stats, e->num_sms, e->compute);
+        CK(cudaMemcpyAsync(&sm->st, s.stats, sizeof(Q18Stats), cudaMemcpyDeviceToHost, e->compute));
+        sync_compute(e);
+        st = sm->st;
+    }
+
+    // a8: ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id — LSD radix sort
+    const unsigned int *perm = nullptr;
+    if (nout > 1) {
+        Q18SortSpec sp;
+        sp.amt_max = st.amt_max;
+        sp.ent_min = st.ent_min;
+        sp.w_min = st.w_min; sp.d_min = st.d_min; sp.o_min = st.o_min;
+        sp.nd = (long long)st.d_max - st.d_min + 1;
+        sp.no = (long long)st.o_max - st.o_min + 1;
+        const unsigned long long nw = (unsigned long long)((long long)st.w_max - st.w_min + 1);
+        sp.bits[0] = bitwidth(nw * (unsigned long long)sp.nd * (unsigned long long)sp.no - 1);
+        sp.bits[1] = bitwidth((unsigned long long)st.ent_max - (unsigned long long)st.ent_min);
+        sp.bits[2] = bitwidth((unsigned long long)st.amt_max - (unsigned long long)st.amt_min);
+        SortScratch ss;
+        ss.max_n = nout;
+        for (int f = 0; f < 3; ++f)
+            ss.key[f] = static_cast<unsigned long long *>(e->arena.get("q18.sk" + std::to_string(f), 8 * nout));
+        ss.idx_a = static_cast<unsigned int *>(e->arena.get("q18.idxa", 4 * nout));
+        ss.idx_b = static_cast<unsigned int *>(e->arena.get("q18.idxb", 4 * nout));
+        const uint64_t tiles = (nout + 8191) / 8192;
+        ss.counts = static_cast<unsigned int *>(e->arena.get("q18.counts", 4ull * 256 * tiles));
+        e->prof.run("q18_sort_keys", [&] { launch_q18_sort_keys(src, nout, sp, ss, e->num_sms, e->compute); });
+        e->prof.run("q18_radix_sort", [&] { perm = radix_sort_fields(nout, sp.bits, ss, e->compute, e->num_sms); });
+    }
+    r->nrows = nout;
+    Q18Cols dst;
+    if (r->on_device) {
+        dst.c_last = static_cast<int32_t *>(result_block(r, 4 * nout));
+        dst.c_id = static_cast<int32_t *>(result_block(r, 4 * nout));
+        dst.o_id = static_cast<int32_t *>(result_block(r, 4 * nout));
+        dst.o_entry_d = static_cast<int64_t *>(result_block(r, 8 * nout));
+        dst.o_ol_cnt = static_cast<int32_t *>(result_block(r, 4 * nout));
+        dst.amount_sum = static_cast<int64_t *>(result_block(r, 8 * nout));
+        dst.o_w_id = static_cast<int32_t *>(result_block(r, 4 * nout));
+        dst.o_d_id = static_cast<int32_t *>(result_block(r, 4 * nout));
+        e->prof.run("q18_permute", [&] { if (nout) launch_q18_permute(src, perm, nout, dst, e->num_sms, e->compute); });
+    } else {
+        Q18Cols sorted = carve_cols(e->arena, "q18.sorted.", nout);
+        e->prof.run("q18_permute", [&] { if (nout) launch_q18_permute(src, perm, nout, sorted, e->num_sms, e->compute); });
+        auto d2h = [&](const void *src_p, size_t es) {
+            void *h = result_block(r, nout * es);
+            if (nout) CK(cudaMemcpyAsync(h, src_p, nout * es, cudaMemcpyDeviceToHost, e->compute));
+            return h;
+        };
+        dst.c_last = static_cast<int32_t *>(d2h(sorted.c_last, 4));
+        dst.c_id = static_cast<int32_t *>(d2h(sorted.c_id, 4));
+        dst.o_id = static_cast<int32_t *>(d2h(sorted.o_id, 4));
+        dst.o_entry_d = static_cast<int64_t *>(d2h(sorted.o_entry_d, 8));
+        dst.o_ol_cnt = static_cast<int32_t *>(d2h(sorted.o_ol_cnt, 4));
+        dst.amount_sum = static_cast<int64_t *>(d2h(sorted.amount_sum, 8));
+        dst.o_w_id = static_cast<int32_t *>(d2h(sorted.o_w_id, 4));
+        dst.o_d_id = static_cast<int32_t *>(d2h(sorted.o_d_id, 4));
+    }
+    CK(cudaGetLastError());
+    CK(cudaEventRecord(e->q_end, e->compute));
+    sync_compute(e);
+    add_col(r, "c_last", H2TAP_I32, dst.c_last);
+    add_col(r, "c_id", H2TAP_I32, dst.c_id);
+    add_col(r, "o_id", H2TAP_I32, dst.o_id);
+    add_col(r, "o_entry_d", H2TAP_I64, dst.o_entry_d);
+    add_col(r, "o_ol_cnt", H2TAP_I32, dst.o_ol_cnt);
+    add_col(r, "amount_sum", H2TAP_I64, dst.amount_sum);
+    add_col(r, "o_w_id", H2TAP_I32, dst.o_w_id);
+    add_col(r, "o_d_id", H2TAP_I32, dst.o_d_id);
+}
+
+// CH-benCHmark constants as int64 µs UTC / cents (R4, R6).
+constexpr int64_t kQ1Cutoff = 1167696000000000LL;   // 2007-01-02 00:00:00
+constexpr int64_t kQ6DLo = 915148800000000LL;       // 1999-01-01 00:00:00
+constexpr int64_t kQ6DHi = 1577836800000000LL;      // 2020-01-01 00:00:00
+constexpr int64_t kQ18Having = 20000;               // 200.00
+
+h2tap_status query_impl(h2tap_engine *e, uint32_t plan, const int64_t *params, uint32_t nparams,
+                        uint32_t flags, h2tap_result **out) {
+    const auto t0 = std::chrono::steady_clock::now();
+    if (!out) return fail(H2TAP_EINVAL, "out is NULL");
+    *out = nullptr;
+    int64_t p[4];
+    uint32_t want;
+    switch (plan) {
+        case H2TAP_Q1: want = 1; p[0] = kQ1Cutoff; break;
+        case H2TAP_Q6: want = 4; p[0] = kQ6DLo; p[1] = kQ6DHi; p[2] = 1; p[3] = 100000; break;
+        case H2TAP_Q18: want = 1; p[0] = kQ18Having; break;
+        default: return fail(H2TAP_EINVAL, "unknown plan id %u", plan);
+    }
+    if (nparams) {
+        if (nparams != want || !params)
+            return fail(H2TAP_EINVAL, "plan %u takes %u params, got %u", plan, want, nparams);
+        std::memcpy(p, params, sizeof(int64_t) * want);
+    }
+    std::lock_guard<std::mutex> g(e->query_mu);
+    CK(cudaSetDevice(e->device));
+    publish_ready(e, false);
+    ViewP v;
+    {
+        std::lock_guard<std::mutex> gv(e->view_mu);
+        v = e->published;
+    }
+    if (!v) return fail(H2TAP_EPLAN, "no snapshot has been published yet");
+    std::unique_ptr<ResultImpl> r(new_result(e, *v, flags & H2TAP_RESULT_DEVICE));
+    e->prof.reset(flags & H2TAP_QUERY_PROFILE, e->compute);
+    const uint64_t launches0 = launches_total();
+    CK(cudaEventRecord(e->q_begin, e->compute));
+    switch (plan) {
+        case H2TAP_Q1: run_q1(e, *v, p, r.get()); break;
+        case H2TAP_Q6: run_q6(e, *v, p, r.get()); break;
+        case H2TAP_Q18: run_q18(e, *v, p, r.get()); break;
+    }
+    float ms = 0;
+    CK(cudaEventElapsedTime(&ms, e->q_begin, e->q_end));
+    r->device_ms = ms;
+    r->kernel_launches = launches_total() - launches0;
+    for (auto &m : e->prof.marks) {
+        float k = 0;
+        CK(cudaEventElapsedTime(&k, m.second.first, m.second.second));
+        r->kname_store.push_back(m.first);
+        r->kms.push_back(k);
+    }
+    r->e2e_ms = std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - t0).count();
+    r->finish();
+    *out = r.release();
+    return H2TAP_OK;
+}
+
+template <class F> h2tap_status guarded(F &&f) {
+    try {
+        return f();
+    } catch (const Fail &x) {
+        return x.st;
+    } catch (const std::bad_alloc &) {
+        return fail(H2TAP_ENOMEM, "host allocation failed");
+    } catch (...) {
+        return fail(H2TAP_EINVAL, "unexpected internal error");
+    }
+}
+
+}  // namespace
+
+// ================================================================ ABI ===
+extern "C" {
+
+h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
+    return guarded([&]() -> h2tap_status {
+        if (!cfg || !out) return fail(H2TAP_EINVAL, "cfg/out is NULL");
+        *out = nullptr;
+        if (cfg->world < 1 || cfg->rank < 0 || cfg->rank >= cfg->world)
+            return fail(H2TAP_EINVAL, "bad rank %d / world %d", cfg->rank, cfg->world);
+        if (cfg->world > 1 && !cfg->nccl_unique_id)
+            return fail(H2TAP_EINVAL, "world > 1 needs an NCCL unique id");
+        int ndev = 0;
+        CK(cudaGetDeviceCount(&ndev));
+        if (cfg->device < 0 || cfg->device >= ndev)
+            return fail(H2TAP_EINVAL, "device %d not present (%d devices)", cfg->device, ndev);
+        std::unique_ptr<h2tap_engine> e(new h2tap_engine());
+        e->device = cfg->device;
+        e->rank = cfg->rank;
+        e->world = cfg->world;
+        CK(cudaSetDevice(e->device));
+        cudaDeviceProp prop;
+        CK(cudaGetDeviceProperties(&prop, e->device));
+        if (prop.major != 10)
+            return fail(H2TAP_ECUDA, "built for sm_100a (B200); device %d is sm_%d%d", e->device,
+                        prop.major, prop.minor);
+        e->num_sms = prop.multiProcessorCount;
+        CK(cudaStreamCreateWithFlags(&e->compute, cudaStreamNonBlocking));
+        CK(cudaStreamCreateWithFlags(&e->copy, cudaStreamNonBlocking));
+        CK(cudaEventCreate(&e->q_begin));
+        CK(cudaEventCreate(&e->q_end));
+        CK(cudaMallocHost(&e->small_host, 256));
+        e->arena.device = e->device;
+        e->host_pool = std::make_shared<BlockPool>(true, e->device);
+        e->dev_pool = std::make_shared<BlockPool>(false, e->device);
+        if (e->world > 1) {
+            ncclUniqueId id;
+            std::memcpy(&id, cfg->nccl_unique_id, sizeof id);
+            NK(ncclCommInitRank(&e->comm, e->world, id, e->rank));
+        }
+        *out = e.release();
+        return H2TAP_OK;
+    });
+}
+
+h2tap_status h2tap_load_snapshot_ex(h2tap_engine *e, const h2tap_table *tables, uint32_t ntables,
+                                    uint64_t epoch, uint32_t flags) {
+    if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
+    return guarded([&] { return load_impl(e, tables, ntables, epoch, flags); });
+}
+
+h2tap_status h2tap_load_snapshot(h2tap_engine *e, const h2tap_table *tables, uint32_t ntables,
+                                 uint64_t epoch) {
+    return h2tap_load_snapshot_ex(e, tables, ntables, epoch, 0);
+}
+
+h2tap_status h2tap_sync(h2tap_engine *e, uint64_t *published_epoch) {
+    if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
+    return guarded([&]() -> h2tap_status {
+        CK(cudaSetDevice(e->device));
+        publish_ready(e, true);
+        std::lock_guard<std::mutex> gv(e->view_mu);
+        if (published_epoch) *published_epoch = e->published ? e->published->epoch : 0;
+        return H2TAP_OK;
+    });
+}
+
+h2tap_status h2tap_run_query_ex(h2tap_engine *e, uint32_t plan_id, const int64_t *params,
+                                uint32_t nparams, uint32_t flags, h2tap_result **out) {
+    if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
+    return guarded([&] { return query_impl(e, plan_id, params, nparams, flags, out); });
+}
+
+h2tap_status h2tap_run_query(h2tap_engine *e, uint32_t plan_id, const int64_t *params,
+                             uint32_t nparams, h2tap_result **out) {
+    return h2tap_run_query_ex(e, plan_id, params, nparams, 0, out);
+}
+
+void h2tap_free(h2tap_result *r) {
+    if (!r) return;
+    delete static_cast<ResultImpl *>(r);
+}
+
+void h2tap_close(h2tap_engine *e) {
+    if (!e) return;
+    cudaSetDevice(e->device);
+    try { publish_ready(e, true); } catch (...) {}
+    cudaStreamSynchronize(e->compute);
+    cudaStreamSynchronize(e->copy);
+    if (e->comm) ncclCommDestroy(e->comm);
+    for (auto &p : e->pending) cudaEventDestroy(p.done);
+    for (int k = 0; k < Staging::kSlots; ++k) {
+        if (e->staging.buf[k]) cudaFreeHost(e->staging.buf[k]);
+        if (e->staging.ev[k]) cudaEventDestroy(e->staging.ev[k]);
+    }
+    for (auto ev : e->prof.pool) cudaEventDestroy(ev);
+    cudaEventDestroy(e->q_begin);
+    cudaEventDestroy(e->q_end);
+    cudaFreeHost(e->small_host);
+    e->published.reset();
+    e->accepted.reset();
+    for (auto &t : e->tables) for (auto &c : t.col) { c.cur.reset(); c.spare.reset(); }
+    e->arena.bufs.clear();
+    cudaStreamDestroy(e->compute);
+    cudaStreamDestroy(e->copy);
+    delete e;
+}
+
+const char *h2tap_last_error(void) { return g_err.c_str(); }
+
+h2tap_status h2tap_nccl_unique_id(void *out128) {
+    if (!out128) return fail(H2TAP_EINVAL, "out is NULL");
+    return guarded([&]() -> h2tap_status {
+        ncclUniqueId id;
+        NK(ncclGetUniqueId(&id));
+        static_assert(sizeof(ncclUniqueId) == 128, "ncclUniqueId is 128 bytes");
+        std::memcpy(out128, &id, sizeof id);
+        return H2TAP_OK;
+    });
+}
+
+h2tap_status h2tap_compute_stream(h2tap_engine *e, void **stream) {
+    if (!e || !stream) return fail(H2TAP_EINVAL, "NULL argument");
+    *stream = e->compute;
+    return H2TAP_OK;
+}
+
+int h2tap_c_last_name(int32_t code, char *buf, size_t buflen) {
+    // TPC-C 4.3.2.3: C_LAST is the concatenation of the syllables of the three digits of code
+    static const char *syl[10] = {"BAR", "OUGHT", "ABLE", "PRI", "PRES",
+                                  "ESE", "ANTI", "CALLY", "ATION", "EING"};
+    if (code < 0 || code > 999 || !buf) return -1;
+    const int n = snprintf(buf, buflen, "%s%s%s", syl[code / 100], syl[(code / 10) % 10], syl[code % 10]);
+    return (n < 0 || (size_t)n >= buflen) ? -1 : n;
+}
+
+}  // extern "C"

@@ -1,0 +1,117 @@
+// kernels.cuh — internal interface between the engine (engine.cu) and the sm_100a kernels.
+// Product code only; never included by oracle/.
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+namespace h2tap {
+
+constexpr int64_t kNullTs = INT64_MIN;  // SQL NULL of ol_delivery_d (R5)
+
+// ----------------------------------------------------------------- Q6 (K1) --
+// revenue = SUM(amount) over rows with d_lo <= delivery < d_hi AND q_lo <= qty <= q_hi.
+// out[0] = revenue, out[1] = qualifying row count. Partials: one {sum,cnt} per block,
+// reduced by the last block to finish (no memset needed; the counter self-resets).
+struct Q6Scratch {
+    long long *block_part;      // [2 * max_blocks]
+    unsigned int *done_counter; // [1], zero-initialised once at allocation
+    long long *out;             // [2]
+};
+int q6_max_blocks(int num_sms);
+void launch_q6(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uint64_t n,
+               int64_t d_lo, int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s,
+               int num_sms, cudaStream_t st);
+
+// ----------------------------------------------------------------- Q1 (K2) --
+// GROUP BY ol_number over rows with delivery > cutoff; per group (count, sum_qty, sum_amount).
+// Keys in [0, kQ1Dense) are aggregated in thread-private shared memory; other keys go through
+// warp-aggregated shared-memory atomics into a per-block hash table, then a global hash table.
+constexpr int kQ1Dense = 16;
+constexpr int kQ1GlobalSlots = 1 << 16;  // max distinct groups per rank
+struct Q1Group { long long key; long long cnt, qty, amt; };  // 32 B, compacted group
+struct Q1Scratch {
+    unsigned long long *dense;   // [kQ1Dense * 3]: cnt, qty, amt per dense key
+    unsigned long long *gtag;    // [kQ1GlobalSlots]: 0 = empty, else (1<<32 | (u32)key)
+    unsigned long long *gacc;    // [kQ1GlobalSlots * 3]
+    unsigned int *flags;         // [1]: bit0 = global table full
+    Q1Group *groups;             // [kQ1GlobalSlots + kQ1Dense] compacted groups
+    unsigned long long *ngroups; // [1]
+    // output (ranked by key)
+    int32_t *o_key; long long *o_qty, *o_amt, *o_cnt; double *o_avg_qty, *o_avg_amt;
+};
+void launch_q1_reset(const Q1Scratch &s, cudaStream_t st);
+void launch_q1(const int32_t *number, const int64_t *deliv, const int32_t *qty,
+               const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int num_sms,
+               cudaStream_t st);
+void launch_q1_compact(const Q1Scratch &s, cudaStream_t st);        // tables -> groups[], ngroups
+void launch_q1_merge(const Q1Group *all, uint64_t n, const Q1Scratch &s, cudaStream_t st);
+void launch_q1_emit(const Q1Scratch &s, uint64_t ngroups, cudaStream_t st);  // rank by key + AVG
+
+// ------------------------------------------------------------ Q18 (K3-K5) --
+struct HtSlot { unsigned long long key; unsigned int row; unsigned int pad; };  // 16 B
+constexpr unsigned long long kEmpty = ~0ull;
+struct Q18Acc { long long sum; unsigned int cnt; unsigned int pad; };          // 16 B
+enum : unsigned int { kErrDupOrders = 1u, kErrDupCustomer = 2u, kErrDomain = 4u };
+
+struct Q18Stats {            // min/max of the sort fields over result rows (atomics)
+    long long amt_min, amt_max, ent_min, ent_max;
+    int w_min, w_max, d_min, d_max, o_min, o_max, pad0, pad1;
+};
+struct Q18Cols {             // SoA result columns
+    int32_t *c_last, *c_id, *o_id, *o_ol_cnt, *o_w_id, *o_d_id;
+    int64_t *o_entry_d, *amount_sum;
+};
+struct Q18Scratch {
+    HtSlot *ht_o; uint64_t cap_o;
+    HtSlot *ht_c; uint64_t cap_c;
+    Q18Acc *acc;             // [n_orders]
+    unsigned int *err;       // [1]
+    unsigned long long *nout;// [1]
+    Q18Stats *stats;         // [1]
+    Q18Cols un;              // unsorted result columns [n_orders]
+};
+void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, cudaStream_t st);
+void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
+                      const int32_t *c_w, const int32_t *c_d, const int32_t *c_id, uint64_t n_c,
+                      const Q18Scratch &s, int num_sms, cudaStream_t st);
+void launch_q18_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
+                      const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
+                      cudaStream_t st);
+void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id,
+                       const int32_t *o_c, const int32_t *o_cnt, const int64_t *o_ent,
+                       uint64_t n_o, const int32_t *c_last, int64_t having,
+                       const Q18Scratch &s, int num_sms, cudaStream_t st);
+void launch_q18_stats(const Q18Cols &cols, uint64_t n, Q18Stats *stats, int num_sms,
+                      cudaStream_t st);  // recompute stats over gathered rows (multi-GPU)
+
+// ------------------------------------------------------------------ sort ---
+// Stable LSD radix sort of a permutation by up to three unsigned key fields (least significant
+// field first), 8-bit digits, only as many passes as each field's bit width needs.
+struct SortScratch {
+    unsigned long long *key[3];  // [n] per field
+    unsigned int *idx_a, *idx_b; // [n]
+    unsigned int *counts;        // [256 * max_tiles]
+    size_t max_n;
+};
+constexpr int kSortItems = 64;                 // items per lane per tile
+constexpr int kSortTile = 32 * kSortItems;     // elements per warp tile
+inline uint64_t sort_tiles(uint64_t n) { return (n + kSortTile - 1) / kSortTile; }
+struct Q18SortSpec {         // host-computed from Q18Stats
+    long long amt_max, ent_min; int w_min, d_min, o_min; long long nd, no;  // dense rowkey
+    int bits[3];             // field 0: rowkey (asc), 1: entry (asc), 2: amount (desc)
+};
+void launch_q18_sort_keys(const Q18Cols &cols, uint64_t n, const Q18SortSpec &spec,
+                          const SortScratch &s, int num_sms, cudaStream_t st);
+// Sorts; returns the buffer holding the final permutation.
+unsigned int *radix_sort_fields(uint64_t n, const int bits[3], const SortScratch &s,
+                                cudaStream_t st, int num_sms);
+void launch_q18_permute(const Q18Cols &src, const unsigned int *perm, uint64_t n,
+                        const Q18Cols &dst, int num_sms, cudaStream_t st);
+
+// ---------------------------------------------------------------- helpers --
+// Every launcher counts the kernels it launches (reported per query as kernel_launches).
+void count_launches(int n);
+uint64_t launches_total();
+void launch_fill_u64(unsigned long long *p, uint64_t n, unsigned long long v, cudaStream_t st);
+
+}  // namespace h2tap

@@ -1,0 +1,453 @@
+// scan_kernels.cu — K1 (CH Q6 fused scan-filter-sum) and K2 (CH Q1 fused scan-filter-group-by)
+// for sm_100a.
+//
+// Paper anchor: the data-parallel archipelago runs OLAP scans over a columnar (DSM) snapshot
+// (Fig. 3); "GPUs coalesce global memory loads ... threads should access
+// memory locations sequentially" (L511-517), which is what DSM buys (L987-990). The paper runs
+// one CUDA kernel per primitive with materialised intermediates and calls that sub-optimal
+// (L527-535) with fusion as future work (L552-554): here each query is ONE fused kernel plus a
+// tiny finaliser, and the scan is HBM-bound (20 B/row for Q6, 24 B/row for Q1).
+#include <cstdint>
+#include <cuda_runtime.h>
+
+#include "kernels.cuh"
+
+namespace h2tap {
+namespace {
+
+constexpr unsigned kFull = 0xffffffffu;
+
+// 128-bit streaming loads: read-only path, do not allocate in L1 (each byte is read once).
+__device__ __forceinline__ longlong2 ld_stream(const longlong2 *p) {
+    longlong2 r;
+    asm volatile("ld.global.nc.L1::no_allocate.v2.s64 {%0, %1}, [%2];"
+                 : "=l"(r.x), "=l"(r.y) : "l"(p));
+    return r;
+}
+__device__ __forceinline__ int4 ld_stream(const int4 *p) {
+    int4 r;
+    asm volatile("ld.global.nc.L1::no_allocate.v4.s32 {%0, %1, %2, %3}, [%4];"
+                 : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w) : "l"(p));
+    return r;
+}
+
+__device__ __forceinline__ long long warp_sum(long long v) {
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(kFull, v, o);
+    return v;
+}
+
+// ================================================================== Q6 ====
+constexpr int kQ6Threads = 256;
+constexpr int kQ6Unroll = 2;  // 4-row vectors per thread per iteration
+
+struct Q6Pred {
+    long long d_lo, d_hi, q_lo, q_hi;
+    // WHERE ol_delivery_d >= d_lo AND ol_delivery_d < d_hi AND ol_quantity BETWEEN q_lo AND q_hi;
+    // a NULL delivery date (INT64_MIN) makes the conjunction UNKNOWN -> row excluded (R5).
+    __device__ __forceinline__ bool operator()(long long d, int q) const {
+        return (d != kNullTs) & (d >= d_lo) & (d < d_hi) & ((long long)q >= q_lo) &
+               ((long long)q <= q_hi);
+    }
+};
+
+__global__ void __launch_bounds__(kQ6Threads)
+q6_kernel(const longlong2 *__restrict__ deliv, const int4 *__restrict__ qty,
+          const longlong2 *__restrict__ amt, uint64_t n, Q6Pred pred,
+          long long *__restrict__ part, unsigned int *__restrict__ counter,
+          long long *__restrict__ out) {
+    long long sum = 0, cnt = 0;
+    const uint64_t nvec = n >> 2;  // 4 rows per vector: 2x16B deliv, 16B qty, 2x16B amount
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+
+    auto row = [&](long long d, int q, long long a) {
+        const bool p = pred(d, q);
+        sum += p ? a : 0;
+        cnt += p;
+    };
+    for (; v + (kQ6Unroll - 1) * stride < nvec; v += kQ6Unroll * stride) {
+        longlong2 d0[kQ6Unroll], d1[kQ6Unroll], a0[kQ6Unroll], a1[kQ6Unroll];
+        int4 q[kQ6Unroll];
+#pragma unroll
+        for (int u = 0; u < kQ6Unroll; ++u) {
+            const uint64_t x = v + u * stride;
+            d0[u] = ld_stream(deliv + 2 * x);
+            d1[u] = ld_stream(deliv + 2 * x + 1);
+            q[u] = ld_stream(qty + x);
+            a0[u] = ld_stream(amt + 2 * x);
+            a1[u] = ld_stream(amt + 2 * x + 1);
+        }
+#pragma unroll
+        for (int u = 0; u < kQ6Unroll; ++u) {
+            row(d0[u].x, q[u].x, a0[u].x);
+            row(d0[u].y, q[u].y, a0[u].y);
+            row(d1[u].x, q[u].z, a1[u].x);
+            row(d1[u].y, q[u].w, a1[u].y);
+        }
+    }
+    for (; v < nvec; v += stride) {
+        const longlong2 d0 = ld_stream(deliv + 2 * v), d1 = ld_stream(deliv + 2 * v + 1);
+        const int4 q = ld_stream(qty + v);
+        const longlong2 a0 = ld_stream(amt + 2 * v), a1 = ld_stream(amt + 2 * v + 1);
+        row(d0.x, q.x, a0.x);
+        row(d0.y, q.y, a0.y);
+        row(d1.x, q.z, a1.x);
+        row(d1.y, q.w, a1.y);
+    }
+    {  // ragged tail: rows [4*nvec, n), at most 3, masked by the visible row count
+        const uint64_t t = 4 * nvec + (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+        if (t < n) {
+            const long long *D = reinterpret_cast<const long long *>(deliv);
+            const int *Q = reinterpret_cast<const int *>(qty);
+            const long long *A = reinterpret_cast<const long long *>(amt);
+            row(D[t], Q[t], A[t]);
+        }
+    }
+
+    // block reduction: warp shuffles -> shared -> warp 0
+    __shared__ long long s_sum[kQ6Threads / 32], s_cnt[kQ6Threads / 32];
+    __shared__ bool s_last;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    sum = warp_sum(sum);
+    cnt = warp_sum(cnt);
+    if (lane == 0) { s_sum[warp] = sum; s_cnt[warp] = cnt; }
+    __syncthreads();
+    if (warp == 0) {
+        sum = lane < kQ6Threads / 32 ? s_sum[lane] : 0;
+        cnt = lane < kQ6Threads / 32 ? s_cnt[lane] : 0;
+        sum = warp_sum(sum);
+        cnt = warp_sum(cnt);
+        if (lane == 0) {
+            part[2 * blockIdx.x] = sum;
+            part[2 * blockIdx.x + 1] = cnt;
+            __threadfence();
+            const unsigned int ticket = atomicAdd(counter, 1u);
+            s_last = ticket == gridDim.x - 1;
+        }
+    }
+    __syncthreads();
+    if (s_last) {  // last block to finish folds all block partials (fixed order, exact ints)
+        __threadfence();
+        long long ts = 0, tc = 0;
+        for (unsigned b = threadIdx.x; b < gridDim.x; b += blockDim.x) {
+            ts += __ldcg(part + 2 * b);
+            tc += __ldcg(part + 2 * b + 1);
+        }
+        ts = warp_sum(ts);
+        tc = warp_sum(tc);
+        if (lane == 0) { s_sum[warp] = ts; s_cnt[warp] = tc; }
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            long long S = 0, C = 0;
+            for (int w = 0; w < kQ6Threads / 32; ++w) { S += s_sum[w]; C += s_cnt[w]; }
+            out[0] = S;
+            out[1] = C;
+            *counter = 0;  // self-reset for the next launch
+        }
+    }
+}
+
+// ================================================================== Q1 ====
+constexpr int kQ1Threads = 256;
+constexpr int kQ1Unroll = 2;   // 4-row vectors per lane per warp iteration
+constexpr int kQ1Sparse = 256; // per-block shared hash slots for keys outside [0, kQ1Dense)
+
+struct Q1Smem {
+    unsigned int cnt[kQ1Dense][kQ1Threads];  // [key][thread]: lane-distinct banks, no conflicts
+    long long qty[kQ1Dense][kQ1Threads];
+    long long amt[kQ1Dense][kQ1Threads];
+    unsigned long long stag[kQ1Sparse];      // 0 = empty, else (1<<32 | (u32)key)
+    unsigned long long sacc[kQ1Sparse][3];
+};
+
+__device__ __forceinline__ unsigned int hash32(unsigned int x) {
+    x ^= x >> 16; x *= 0x7feb352dU; x ^= x >> 15; x *= 0x846ca68bU; x ^= x >> 16;
+    return x;
+}
+
+__device__ void q1_global_add(const Q1Scratch &g, unsigned long long tag, unsigned long long c,
+                              long long q, long long a) {
+    unsigned int h = hash32((unsigned int)tag) & (kQ1GlobalSlots - 1);
+    for (int p = 0; p < kQ1GlobalSlots; ++p) {
+        const unsigned long long prev = atomicCAS(g.gtag + h, 0ull, tag);
+        if (prev == 0ull || prev == tag) {
+            atomicAdd(g.gacc + 3 * h + 0, c);
+            atomicAdd(g.gacc + 3 * h + 1, (unsigned long long)q);
+            atomicAdd(g.gacc + 3 * h + 2, (unsigned long long)a);
+            return;
+        }
+        h = (h + 1) & (kQ1GlobalSlots - 1);
+    }
+    atomicOr(g.flags, 1u);  // more distinct groups than kQ1GlobalSlots: reported as ENOMEM
+}
+
+__device__ void q1_sparse_add(Q1Smem &sm, const Q1Scratch &g, int key, unsigned long long c,
+                              long long q, long long a) {
+    const unsigned long long tag = (1ull << 32) | (unsigned int)key;
+    unsigned int h = hash32((unsigned int)key) & (kQ1Sparse - 1);
+    for (int p = 0; p < kQ1Sparse; ++p) {
+        const unsigned long long prev = atomicCAS(&sm.stag[h], 0ull, tag);
+        if (prev == 0ull || prev == tag) {
+            atomicAdd(&sm.sacc[h][0], c);
+            atomicAdd(&sm.sacc[h][1], (unsigned long long)q);
+            atomicAdd(&sm.sacc[h][2], (unsigned long long)a);
+            return;
+        }
+        h = (h + 1) & (kQ1Sparse - 1);
+    }
+    q1_global_add(g, tag, c, q, a);  // block table full: go straight to the global table
+}
+
+// Warp-aggregated shared-memory atomics: lanes with the same key are grouped (one ballot per
+// distinct key present in the warp), their values are reduced with shuffles, and only the
+// group leader touches the hash table. Called convergently by all 32 lanes.
+__device__ __forceinline__ void q1_sparse_warp(Q1Smem &sm, const Q1Scratch &g, bool need, int key,
+                                               long long q, long long a) {
+    const int lane = threadIdx.x & 31;
+    unsigned int pend = __ballot_sync(kFull, need);
+    while (pend) {
+        const int leader = __ffs(pend) - 1;
+        const int lk = __shfl_sync(kFull, key, leader);
+        const bool in = need && key == lk;
+        const unsigned int grp = __ballot_sync(kFull, in);
+        const long long qs = warp_sum(in ? q : 0);
+        const long long as = warp_sum(in ? a : 0);
+        if (lane == leader) q1_sparse_add(sm, g, lk, __popc(grp), qs, as);
+        need = need && !in;
+        pend &= ~grp;
+    }
+}
+
+__global__ void __launch_bounds__(kQ1Threads, 2)
+q1_kernel(const int4 *__restrict__ number, const longlong2 *__restrict__ deliv,
+          const int4 *__restrict__ qty, const longlong2 *__restrict__ amt, uint64_t n,
+          long long cutoff, Q1Scratch g) {
+    extern __shared__ __align__(16) unsigned char smem_raw[];
+    Q1Smem &sm = *reinterpret_cast<Q1Smem *>(smem_raw);
+    const int tid = threadIdx.x, lane = tid & 31;
+#pragma unroll
+    for (int k = 0; k < kQ1Dense; ++k) { sm.cnt[k][tid] = 0; sm.qty[k][tid] = 0; sm.amt[k][tid] = 0; }
+    for (int s = tid; s < kQ1Sparse; s += kQ1Threads) {
+        sm.stag[s] = 0; sm.sacc[s][0] = 0; sm.sacc[s][1] = 0; sm.sacc[s][2] = 0;
+    }
+    if (blockIdx.x == 0 && tid == 0) *g.ngroups = 0;  // consumed by q1_compact (stream-ordered)
+    __syncthreads();
+
+    // WHERE ol_delivery_d > cutoff (NULL -> UNKNOWN -> excluded), GROUP BY ol_number
+    auto row = [&](bool valid, int key, long long d, int q, long long a, bool &sparse) {
+        const bool pass = valid & (d != kNullTs) & (d > cutoff);
+        sparse = pass & ((unsigned)key >= (unsigned)kQ1Dense);
+        if (pass & ((unsigned)key < (unsigned)kQ1Dense)) {  // thread-private dense slot
+            sm.cnt[key][tid] += 1;
+            sm.qty[key][tid] += q;
+            sm.amt[key][tid] += a;
+        }
+    };
+
+    const uint64_t nvec = n >> 2;
+    const uint64_t gwarp = ((uint64_t)blockIdx.x * kQ1Threads + tid) >> 5;
+    const uint64_t nwarps = ((uint64_t)gridDim.x * kQ1Threads) >> 5;
+    // warp-uniform trip count so that ballots in the sparse path are convergent
+    for (uint64_t base = gwarp * 32 * kQ1Unroll; base < nvec; base += nwarps * 32 * kQ1Unroll) {
+        int4 nb[kQ1Unroll], qv[kQ1Unroll];
+        longlong2 d0[kQ1Unroll], d1[kQ1Unroll], a0[kQ1Unroll], a1[kQ1Unroll];
+        bool ok[kQ1Unroll];
+#pragma unroll
+        for (int u = 0; u < kQ1Unroll; ++u) {
+            const uint64_t x = base + u * 32 + lane;
+            ok[u] = x < nvec;
+            if (ok[u]) {
+                nb[u] = ld_stream(number + x);
+                d0[u] = ld_stream(deliv + 2 * x);
+                d1[u] = ld_stream(deliv + 2 * x + 1);
+                qv[u] = ld_stream(qty + x);
+                a0[u] = ld_stream(amt + 2 * x);
+                a1[u] = ld_stream(amt + 2 * x + 1);
+            } else {
+                nb[u] = make_int4(0, 0, 0, 0); qv[u] = nb[u];
+                d0[u] = make_longlong2(kNullTs, kNullTs); d1[u] = d0[u];
+                a0[u] = make_longlong2(0, 0); a1[u] = a0[u];
+            }
+        }
+        bool sp[kQ1Unroll][4];
+#pragma unroll
+        for (int u = 0; u < kQ1Unroll; ++u) {
+            row(ok[u], nb[u].x, d0[u].x, qv[u].x, a0[u].x, sp[u][0]);
+            row(ok[u], nb[u].y, d0[u].y, qv[u].y, a0[u].y, sp[u][1]);
+            row(ok[u], nb[u].z, d1[u].x, qv[u].z, a1[u].x, sp[u][2]);
+            row(ok[u], nb[u].w, d1[u].y, qv[u].w, a1[u].y, sp[u][3]);
+        }
+        bool any = false;
+#pragma unroll
+        for (int u = 0; u < kQ1Unroll; ++u) any |= sp[u][0] | sp[u][1] | sp[u][2] | sp[u][3];
+        if (__any_sync(kFull, any)) {  // rare for TPC-C data (ol_number in 1..15)
+#pragma unroll
+            for (int u = 0; u < kQ1Unroll; ++u) {
+                q1_sparse_warp(sm, g, sp[u][0], nb[u].x, qv[u].x, a0[u].x);
+                q1_sparse_warp(sm, g, sp[u][1], nb[u].y, qv[u].y, a0[u].y);
+                q1_sparse_warp(sm, g, sp[u][2], nb[u].z, qv[u].z, a1[u].x);
+                q1_sparse_warp(sm, g, sp[u][3], nb[u].w, qv[u].w, a1[u].y);
+            }
+        }
+    }
+    if (blockIdx.x == 0 && tid < 32) {  // ragged tail rows [4*nvec, n) (<= 3), warp 0 of block 0
+        const uint64_t t = 4 * nvec + lane;
+        const bool valid = t < n;
+        const int *N = reinterpret_cast<const int *>(number);
+        const long long *D = reinterpret_cast<const long long *>(deliv);
+        const int *Q = reinterpret_cast<const int *>(qty);
+        const long long *A = reinterpret_cast<const long long *>(amt);
+        const int key = valid ? N[t] : 0;
+        const long long d = valid ? D[t] : kNullTs;
+        const int q = valid ? Q[t] : 0;
+        const long long a = valid ? A[t] : 0;
+        bool sparse;
+        row(valid, key, d, q, a, sparse);
+        q1_sparse_warp(sm, g, sparse, key, q, a);
+    }
+    __syncthreads();
+
+    // merge: dense keys, one warp per key, one global atomic per (key, accumulator) per block
+    const int warp = tid >> 5;
+    for (int k = warp; k < kQ1Dense; k += kQ1Threads / 32) {
+        long long c = 0, q = 0, a = 0;
+        for (int t = lane; t < kQ1Threads; t += 32) { c += sm.cnt[k][t]; q += sm.qty[k][t]; a += sm.amt[k][t]; }
+        c = warp_sum(c); q = warp_sum(q); a = warp_sum(a);
+        if (lane == 0 && c) {
+            atomicAdd(g.dense + 3 * k + 0, (unsigned long long)c);
+            atomicAdd(g.dense + 3 * k + 1, (unsigned long long)q);
+            atomicAdd(g.dense + 3 * k + 2, (unsigned long long)a);
+        }
+    }
+    for (int s = tid; s < kQ1Sparse; s += kQ1Threads)
+        if (sm.stag[s]) q1_global_add(g, sm.stag[s], sm.sacc[s][0], (long long)sm.sacc[s][1],
+                                      (long long)sm.sacc[s][2]);
+}
+
+// Collect the dense and global tables into groups[] and clear them for the next query.
+__global__ void q1_compact_kernel(Q1Scratch g) {
+    const uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    if (i < (uint64_t)kQ1Dense) {
+        const unsigned long long c = g.dense[3 * i];
+        if (c) {
+            const unsigned long long p = atomicAdd(g.ngroups, 1ull);
+            g.groups[p] = Q1Group{(long long)i, (long long)c, (long long)g.dense[3 * i + 1],
+                                  (long long)g.dense[3 * i + 2]};
+            g.dense[3 * i] = g.dense[3 * i + 1] = g.dense[3 * i + 2] = 0;
+        }
+    }
+    if (i < (uint64_t)kQ1GlobalSlots) {
+        const unsigned long long tag = g.gtag[i];
+        if (tag) {
+            const unsigned long long p = atomicAdd(g.ngroups, 1ull);
+            g.groups[p] = Q1Group{(long long)(int)(unsigned int)tag, (long long)g.gacc[3 * i],
+                                  (long long)g.gacc[3 * i + 1], (long long)g.gacc[3 * i + 2]};
+            g.gtag[i] = 0;
+            g.gacc[3 * i] = g.gacc[3 * i + 1] = g.gacc[3 * i + 2] = 0;
+        }
+    }
+}
+
+// Multi-GPU: fold gathered per-rank groups into the (clean) global table.
+__global__ void q1_merge_kernel(const Q1Group *__restrict__ all, uint64_t n, Q1Scratch g) {
+    const uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    if (i == 0) *g.ngroups = 0;
+    if (i < n) {
+        const Q1Group x = all[i];
+        q1_global_add(g, (1ull << 32) | (unsigned int)(int)x.key, (unsigned long long)x.cnt, x.qty,
+                      x.amt);
+    }
+}
+
+// ORDER BY ol_number: keys are distinct, so each group's output position is its rank
+// (number of smaller keys). AVG = SUM / COUNT in IEEE double, money / 100 (R7).
+__global__ void q1_emit_kernel(Q1Scratch g, uint64_t ng) {
+    __shared__ long long tile[1024];
+    const uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    const long long mine = i < ng ? g.groups[i].key : 0;
+    uint64_t rank = 0;
+    for (uint64_t t0 = 0; t0 < ng; t0 += 1024) {
+        for (uint64_t t = threadIdx.x; t < 1024 && t0 + t < ng; t += blockDim.x)
+            tile[t] = g.groups[t0 + t].key;
+        __syncthreads();
+        const uint64_t lim = ng - t0 < 1024 ? ng - t0 : 1024;
+        for (uint64_t t = 0; t < lim; ++t) rank += tile[t] < mine;
+        __syncthreads();
+    }
+    if (i < ng) {
+        const Q1Group x = g.groups[i];
+        g.o_key[rank] = (int32_t)x.key;
+        g.o_qty[rank] = x.qty;
+        g.o_amt[rank] = x.amt;
+        g.o_cnt[rank] = x.cnt;
+        g.o_avg_qty[rank] = (double)x.qty / (double)x.cnt;
+        g.o_avg_amt[rank] = ((double)x.amt / (double)x.cnt) / 100.0;
+    }
+}
+
+}  // namespace
+
+// ------------------------------------------------------------------ launchers --
+int q6_max_blocks(int num_sms) { return num_sms * 8; }
+
+void launch_q6(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uint64_t n,
+               int64_t d_lo, int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s,
+               int num_sms, cudaStream_t st) {
+    static int occ = 0;
+    if (!occ) cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, q6_kernel, kQ6Threads, 0);
+    int per_sm = occ < 8 ? (occ > 0 ? occ : 1) : 8;
+    uint64_t want = ((n >> 2) + kQ6Threads - 1) / kQ6Threads;
+    uint64_t grid = (uint64_t)num_sms * per_sm;
+    if (want < grid) grid = want ? want : 1;
+    q6_kernel<<<(unsigned)grid, kQ6Threads, 0, st>>>(
+        reinterpret_cast<const longlong2 *>(deliv), reinterpret_cast<const int4 *>(qty),
+        reinterpret_cast<const longlong2 *>(amt), n, Q6Pred{d_lo, d_hi, q_lo, q_hi},
+        s.block_part, s.done_counter, s.out);
+        count_launches(1);
+}
+
+void launch_q1_reset(const Q1Scratch &s, cudaStream_t st) {
+    cudaMemsetAsync(s.dense, 0, sizeof(unsigned long long) * kQ1Dense * 3, st);
+    cudaMemsetAsync(s.gtag, 0, sizeof(unsigned long long) * kQ1GlobalSlots, st);
+    cudaMemsetAsync(s.gacc, 0, sizeof(unsigned long long) * kQ1GlobalSlots * 3, st);
+    cudaMemsetAsync(s.flags, 0, sizeof(unsigned int), st);
+    cudaMemsetAsync(s.ngroups, 0, sizeof(unsigned long long), st);
+}
+
+void launch_q1(const int32_t *number, const int64_t *deliv, const int32_t *qty,
+               const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int num_sms,
+               cudaStream_t st) {
+    static bool init = false;
+    if (!init) {
+        cudaFuncSetAttribute(q1_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             (int)sizeof(Q1Smem));
+        init = true;
+    }
+    uint64_t want = ((n >> 2) + kQ1Threads - 1) / kQ1Threads;
+    uint64_t grid = (uint64_t)num_sms * 2;
+    if (want < grid) grid = want ? want : 1;
+    q1_kernel<<<(unsigned)grid, kQ1Threads, sizeof(Q1Smem), st>>>(
+        reinterpret_cast<const int4 *>(number), reinterpret_cast<const longlong2 *>(deliv),
+        reinterpret_cast<const int4 *>(qty), reinterpret_cast<const longlong2 *>(amt), n, cutoff,
+        s);
+        count_launches(1);
+}
+
+void launch_q1_compact(const Q1Scratch &s, cudaStream_t st) {
+    q1_compact_kernel<<<kQ1GlobalSlots / 256, 256, 0, st>>>(s);
+    count_launches(1);
+}
+
+void launch_q1_merge(const Q1Group *all, uint64_t n, const Q1Scratch &s, cudaStream_t st) {
+    q1_merge_kernel<<<(unsigned)((n + 255) / 256 + 1), 256, 0, st>>>(all, n, s);
+    count_launches(1);
+}
+
+void launch_q1_emit(const Q1Scratch &s, uint64_t ngroups, cudaStream_t st) {
+    if (!ngroups) return;
+    q1_emit_kernel<<<(unsigned)((ngroups + 255) / 256), 256, 0, st>>>(s, ngroups);
+    count_launches(1);
+}
+
+}  // namespace h2tap

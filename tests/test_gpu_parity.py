@@ -1,0 +1,378 @@
+"""GPU parity: the CUDA path, called through the C ABI, against the CPU oracle on the same
+seeded inputs (``-m gpu``; needs a B200).
+
+Bars (BASELINE.json north_star): sums, counts, keys and row sets bit-exact; AVG within relative
+1e-9 (we in fact require bit-equality, both sides compute (double)sum/(double)count the same way,
+and fall back to 1e-9 only in the assertion helper); Q18 rows in the exact ORDER BY order
+(the tie-break makes the order total, R11).
+"""
+import math
+
+import numpy as np
+import pytest
+
+import chgen
+import oracle
+from chref import (Q1_CUTOFF, Q6_D_HI, Q6_D_LO, Q6_Q_HI, Q6_Q_LO, Q18_HAVING, golden, iso_us)
+
+pytestmark = pytest.mark.gpu
+
+Q18_NAMES = ["c_last", "c_id", "o_id", "o_entry_d", "o_ol_cnt", "amount_sum", "o_w_id", "o_d_id"]
+Q1_NAMES = ["ol_number", "sum_qty", "sum_amount", "avg_qty", "avg_amount", "count_order"]
+
+
+@pytest.fixture(scope="module")
+def h():
+    import paper_conf_cidr_appuswamykpa17_b200 as mod
+    return mod
+
+
+@pytest.fixture(scope="module")
+def eng(h):
+    e = h.h2tap_open(0)
+    yield e
+    h.h2tap_close(e)
+
+
+class Loader:
+    """Loads a whole table set as one new epoch (full reload) and runs queries."""
+
+    def __init__(self, h, e):
+        self.h, self.e, self.epoch = h, e, 0
+
+    def load(self, tables, flags=0):
+        self.epoch += 1
+        self.h.h2tap_load_snapshot(self.e, self.h.hot_path_tables(tables), self.epoch, flags=flags)
+
+    def q(self, plan, params=None, flags=0):
+        r = self.h.h2tap_run_query(self.e, plan, params, flags=flags)
+        try:
+            out = r.to_numpy()
+            out["_nulls"] = dict(r.nulls)
+            out["_meta"] = (r.epoch, r.nrows, r.rows_scanned)
+        finally:
+            r.free()
+        return out
+
+
+@pytest.fixture(scope="module")
+def L(h, eng):
+    return Loader(h, eng)
+
+
+def assert_q6(got, want):
+    assert got["count_rows"][0] == want["count"]
+    if want["revenue"] is None:
+        assert got["_nulls"]["revenue"][0] == 1
+    else:
+        assert got["_nulls"]["revenue"][0] == 0
+        assert got["revenue"][0] == want["revenue"]
+
+
+def assert_q1(got, want):
+    for k in ("ol_number", "sum_qty", "sum_amount", "count_order"):
+        assert np.array_equal(got[k], want[k]), k
+    for k in ("avg_qty", "avg_amount"):
+        assert len(got[k]) == len(want[k])
+        for a, b in zip(got[k].tolist(), want[k].tolist()):
+            assert math.isclose(a, b, rel_tol=1e-9, abs_tol=0.0), (k, a, b)
+
+
+def assert_q18(got, want):
+    for k in Q18_NAMES:
+        assert np.array_equal(got[k], want[k]), k
+
+
+def run_all(L, t, rng=None, n_rand=2):
+    L.load(t)
+    assert_q6(L.q(6, [Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI]), oracle.q6(t, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))
+    assert_q6(L.q(6), oracle.q6(t, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))  # CH defaults in the library
+    assert_q1(L.q(1, [Q1_CUTOFF]), oracle.q1(t, Q1_CUTOFF))
+    assert_q1(L.q(1), oracle.q1(t, Q1_CUTOFF))
+    assert_q18(L.q(18, [Q18_HAVING]), oracle.q18(t, Q18_HAVING))
+    assert_q18(L.q(18), oracle.q18(t, Q18_HAVING))
+    rng = rng or np.random.default_rng(0)
+    for _ in range(n_rand):
+        d_lo = int(rng.integers(chgen.TS_1995, chgen.TS_2025))
+        d_hi = int(rng.integers(d_lo, chgen.TS_2025 + 31 * chgen.DAY_US))
+        q_lo, q_hi = int(rng.integers(0, 6)), int(rng.integers(4, 12))
+        assert_q6(L.q(6, [d_lo, d_hi, q_lo, q_hi]), oracle.q6(t, d_lo, d_hi, q_lo, q_hi))
+        cut = int(rng.integers(chgen.TS_1995, chgen.TS_2025))
+        assert_q1(L.q(1, [cut]), oracle.q1(t, cut))
+        thr = int(rng.integers(-10, 8_000_000))
+        assert_q18(L.q(18, [thr]), oracle.q18(t, thr))
+
+
+# ----------------------------------------------------------------- cases --
+def test_golden_fixture(L):
+    t, exp = golden()
+    L.load(t)
+    for case in exp["q6"]:
+        d_lo, d_hi, q_lo, q_hi = case["params"]
+        got = L.q(6, [iso_us(d_lo), iso_us(d_hi), q_lo, q_hi])
+        assert_q6(got, {"revenue": case["revenue"], "count": case["count"]})
+    for case in exp["q1"]:
+        got = L.q(1, [iso_us(case["params"][0])])
+        assert got["ol_number"].tolist() == [r["ol_number"] for r in case["rows"]]
+        assert got["sum_amount"].tolist() == [r["sum_amount"] for r in case["rows"]]
+        assert got["avg_amount"].tolist() == [r["avg_amount"] for r in case["rows"]]
+    for case in exp["q18"]:
+        got = L.q(18, case["params"])
+        assert got["amount_sum"].tolist() == [r["amount_sum"] for r in case["rows"]]
+        assert got["o_entry_d"].tolist() == [iso_us(r["o_entry_d"]) for r in case["rows"]]
+        assert got["c_last"].tolist() == [r["c_last"] for r in case["rows"]]
+
+
+@pytest.mark.parametrize("W,mode,seed", [(1, "spread", 1), (3, "spread", 2), (2, "strict", 3)])
+def test_parity_small(L, W, mode, seed):
+    run_all(L, chgen.generate(1, W + 1, seed=seed, mode=mode), np.random.default_rng(seed))
+
+
+@pytest.mark.parametrize("n", [0, 1, 2, 3, 4, 5, 7, 127, 128, 129, 4097, 100_003])
+def test_ragged_order_line(L, n):
+    """Row counts that leave a ragged tail after 4-row vectors / 32-row warps / tiles."""
+    t = chgen.generate(1, 2, seed=5)
+    t["order_line"] = {k: v[:n].copy() for k, v in t["order_line"].items()}
+    run_all(L, t, n_rand=1)
+
+
+def test_empty_tables(L):
+    t = chgen.generate(1, 1, seed=1)  # zero warehouses: every table empty
+    L.load(t)
+    got = L.q(6)
+    assert got["_nulls"]["revenue"][0] == 1 and got["count_rows"][0] == 0
+    assert len(L.q(1)["ol_number"]) == 0
+    assert len(L.q(18, [-100])["o_id"]) == 0
+
+
+def test_q1_sparse_group_keys(L):
+    """Keys outside the dense range [0,16): warp-aggregated shared/global hash path."""
+    t = chgen.generate(1, 3, seed=8)
+    ol = t["order_line"]
+    rng = np.random.default_rng(8)
+    n = len(ol["ol_number"])
+    keys = ol["ol_number"].copy()
+    pick = rng.random(n) < 0.5
+    keys[pick] = rng.integers(-3000, 3000, size=int(pick.sum()), dtype=np.int32)
+    keys[:1000] = 2**31 - 1            # long runs of one sparse key
+    keys[1000:1500] = -(2**31)
+    ol["ol_number"] = keys
+    L.load(t)
+    for cut in (Q1_CUTOFF, chgen.TS_1995):
+        assert_q1(L.q(1, [cut]), oracle.q1(t, cut))
+
+
+def test_q6_quantity_and_null_edges(L):
+    t = chgen.generate(1, 2, seed=4)
+    L.load(t)
+    i64 = np.iinfo(np.int64)
+    for p in ([i64.min, i64.max, i64.min, i64.max],      # NULL dates must still be excluded
+              [i64.min + 1, i64.max, 0, 0],              # no quantity 0 -> NULL revenue
+              [Q6_D_LO, Q6_D_LO, 1, 10],                 # empty date window
+              [Q6_D_LO, Q6_D_HI, 10, 1]):                # inverted BETWEEN
+        assert_q6(L.q(6, p), oracle.q6(t, *p))
+
+
+def test_q18_join_edges(L):
+    """Orphan lines, orders without lines, customers missing, negative HAVING."""
+    t = chgen.generate(1, 2, seed=6)
+    ol, o, c = t["order_line"], t["orders"], t["customer"]
+    ol["ol_o_id"][:50] = 7777                      # orphan lines
+    keep = np.ones(len(c["c_id"]), bool)
+    keep[::7] = False                              # drop every 7th customer
+    t["customer"] = {k: v[keep].copy() for k, v in c.items()}
+    mask = o["o_id"] % 11 != 0                     # orders without some rows
+    t["orders"] = {k: v[mask].copy() for k, v in o.items()}
+    L.load(t)
+    for thr in (-1, 0, Q18_HAVING, 4_000_000):
+        assert_q18(L.q(18, [thr]), oracle.q18(t, thr))
+
+
+def test_q18_ties_use_full_order(L):
+    """Equal amount_sum and o_entry_d: the (w, d, o) tie-break decides (R11)."""
+    t = chgen.generate(1, 3, seed=9)
+    t["order_line"]["ol_amount"][:] = 1000
+    t["orders"]["o_entry_d"][:] = chgen.LOAD_TS
+    L.load(t)
+    for thr in (0, 6000):
+        assert_q18(L.q(18, [thr]), oracle.q18(t, thr))
+
+
+def test_q18_duplicate_key_rejected(h, L):
+    t = chgen.generate(1, 2, seed=2)
+    o = t["orders"]
+    for k in o:
+        o[k] = np.concatenate([o[k], o[k][:1]])
+    L.load(t)
+    with pytest.raises(h.H2tapError) as ei:
+        L.q(18)
+    assert ei.value.status == h.H2TAP_EDUPKEY
+    assert_q6(L.q(6), oracle.q6(t, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))  # engine still usable
+
+
+def test_device_resident_results(h, L):
+    t = chgen.generate(1, 3, seed=12)
+    L.load(t)
+    assert_q18(L.q(18, flags=h.H2TAP_RESULT_DEVICE), oracle.q18(t, Q18_HAVING))
+    assert_q1(L.q(1, flags=h.H2TAP_RESULT_DEVICE | h.H2TAP_QUERY_PROFILE), oracle.q1(t, Q1_CUTOFF))
+
+
+def test_profile_reports_kernels(h, eng, L):
+    t = chgen.generate(1, 2, seed=3)
+    L.load(t)
+    r = h.h2tap_run_query(eng, h.H2TAP_Q18, flags=h.H2TAP_QUERY_PROFILE)
+    names = [k for k, _ in r.kernels]
+    assert {"q18_build", "q18_probe_groupjoin", "q18_having_compact", "q18_radix_sort"} <= set(names)
+    assert all(ms >= 0 for _, ms in r.kernels) and r.device_ms > 0
+    r.free()
+
+
+# ------------------------------------------------------- snapshot semantics --
+def test_snapshot_epochs_append_and_errors(h):
+    """a1: append-only refresh, epoch monotonicity, shape errors, async publish."""
+    e = h.h2tap_open(0)
+    try:
+        base = chgen.generate(1, 3, seed=21)
+        cols = h.hot_path_tables(base)
+        h.h2tap_load_snapshot(e, cols, 10)
+        r = h.h2tap_run_query(e, h.H2TAP_Q18)
+        assert r.epoch == 10 and r.rows_scanned == len(base["order_line"]["ol_w_id"])
+        r.free()
+        with pytest.raises(h.H2tapError) as ei:
+            h.h2tap_load_snapshot(e, cols, 10)
+        assert ei.value.status == h.H2TAP_ESTALE
+        # NewOrder delta appended at epoch 11 (host row store -> columns -> H2D delta only)
+        st = chgen.NewOrderState(1, 3)
+        delta = chgen.neworder_delta(st, 300, seed=21, batch=0)
+        n_ol = len(base["order_line"]["ol_w_id"])
+        n_o = len(base["orders"]["o_id"])
+        d = h.hot_path_tables({"order_line": delta["order_line"], "orders": delta["orders"],
+                               "customer": {k: v[:0] for k, v in base["customer"].items()}})
+        d.pop("customer")
+        with pytest.raises(h.H2tapError) as ei:  # wrong first_row
+            h.h2tap_load_snapshot(e, d, 11, full_reload=False, first_row={"order_line": n_ol - 1, "orders": n_o})
+        assert ei.value.status == h.H2TAP_ESHAPE
+        h.h2tap_load_snapshot(e, d, 11, full_reload=False, first_row={"order_line": n_ol, "orders": n_o},
+                              flags=h.H2TAP_LOAD_ASYNC)
+        assert h.h2tap_sync(e) == 11
+        merged = {t: {k: np.concatenate([base[t][k], delta[t][k]]) for k in base[t]}
+                  for t in ("order_line", "orders")}
+        merged["customer"] = base["customer"]
+        r = h.h2tap_run_query(e, h.H2TAP_Q18, [-1])
+        got = r.to_numpy()
+        assert r.epoch == 11 and r.rows_scanned == n_ol + len(delta["order_line"]["ol_w_id"])
+        r.free()
+        assert_q18(got, oracle.q18(merged, -1))
+        # Q6/Q1 unchanged by NewOrder rows (NULL delivery dates, R16) but see the new epoch
+        r6 = h.h2tap_run_query(e, h.H2TAP_Q6)
+        assert r6.to_numpy()["count_rows"][0] == oracle.q6(base, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI)["count"]
+        r6.free()
+        # a result from an earlier epoch stays valid after a full reload
+        old = h.h2tap_run_query(e, h.H2TAP_Q1)
+        h.h2tap_load_snapshot(e, h.hot_path_tables(chgen.generate(1, 2, seed=99)), 12)
+        assert_q1(old.to_numpy(), oracle.q1(merged, Q1_CUTOFF))
+        old.free()
+        with pytest.raises(h.H2tapError) as ei:
+            h.h2tap_run_query(e, h.H2TAP_Q6, [1, 2])
+        assert ei.value.status == h.H2TAP_EINVAL
+    finally:
+        h.h2tap_close(e)
+
+
+def test_concurrent_refresh_and_queries(h):
+    """Queries running while another thread appends see a consistent published epoch."""
+    import threading
+    e = h.h2tap_open(0)
+    try:
+        base = chgen.generate(1, 3, seed=31)
+        h.h2tap_load_snapshot(e, h.hot_path_tables(base), 1)
+        st = chgen.NewOrderState(1, 3)
+        deltas = [chgen.neworder_delta(st, 50, seed=31, batch=b) for b in range(6)]
+        errors = []
+
+        def refresher():
+            try:
+                n_ol, n_o = len(base["order_line"]["ol_w_id"]), len(base["orders"]["o_id"])
+                for b, d in enumerate(deltas):
+                    dd = h.hot_path_tables({**d, "customer": base["customer"]})
+                    dd.pop("customer")
+                    h.h2tap_load_snapshot(e, dd, 2 + b, full_reload=False,
+                                          first_row={"order_line": n_ol, "orders": n_o},
+                                          flags=h.H2TAP_LOAD_ASYNC)
+                    n_ol += len(d["order_line"]["ol_w_id"])
+                    n_o += len(d["orders"]["o_id"])
+            except Exception as x:  # pragma: no cover
+                errors.append(x)
+
+        th = threading.Thread(target=refresher)
+        th.start()
+        seen = []
+        for _ in range(20):
+            r = h.h2tap_run_query(e, h.H2TAP_Q18, [-1])
+            seen.append((r.epoch, r.nrows, r.rows_scanned))
+            r.free()
+        th.join()
+        assert not errors
+        h.h2tap_sync(e)
+        # each observed epoch must be exactly the base plus the first (epoch-1) deltas
+        for ep, nrows, scanned in seen:
+            k = ep - 1
+            want_rows = len(base["orders"]["o_id"]) + sum(len(d["orders"]["o_id"]) for d in deltas[:k])
+            want_scan = len(base["order_line"]["ol_w_id"]) + sum(len(d["order_line"]["ol_w_id"]) for d in deltas[:k])
+            assert (nrows, scanned) == (want_rows, want_scan), (ep, nrows, scanned)
+        assert [s[0] for s in seen] == sorted(s[0] for s in seen)
+    finally:
+        h.h2tap_close(e)
+
+
+# ------------------------------------------------------ re-partition on 1 GPU --
+def test_repartition_matches_whole(h):
+    """Per-shard results (the per-rank partials of a multi-GPU run) merged = whole."""
+    W, k = 6, 3
+    whole = chgen.generate(1, W + 1, seed=41)
+    rev = cnt = 0
+    q1m = {}
+    rows = []
+    for lo, hi in chgen.warehouse_ranges(W, k):
+        e = h.h2tap_open(0)
+        try:
+            part = chgen.generate(lo, hi, seed=41)
+            h.h2tap_load_snapshot(e, h.hot_path_tables(part), 1)
+            r = h.h2tap_run_query(e, h.H2TAP_Q6); x = r.to_numpy(); r.free()
+            rev += int(x["revenue"][0]); cnt += int(x["count_rows"][0])
+            r = h.h2tap_run_query(e, h.H2TAP_Q1); x = r.to_numpy(); r.free()
+            for i, n in enumerate(x["ol_number"].tolist()):
+                m = q1m.setdefault(n, [0, 0, 0])
+                m[0] += int(x["sum_qty"][i]); m[1] += int(x["sum_amount"][i]); m[2] += int(x["count_order"][i])
+            r = h.h2tap_run_query(e, h.H2TAP_Q18); x = r.to_numpy(); r.free()
+            rows += list(zip(*[x[c].tolist() for c in Q18_NAMES]))
+        finally:
+            h.h2tap_close(e)
+    w6 = oracle.q6(whole, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI)
+    assert (rev, cnt) == (w6["revenue"], w6["count"])
+    w1 = oracle.q1(whole, Q1_CUTOFF)
+    for i, n in enumerate(w1["ol_number"].tolist()):
+        assert q1m[n] == [int(w1["sum_qty"][i]), int(w1["sum_amount"][i]), int(w1["count_order"][i])]
+    w18 = oracle.q18(whole, Q18_HAVING)
+    assert sorted(rows) == sorted(zip(*[w18[c].tolist() for c in Q18_NAMES]))
+
+
+# --------------------------------------------- full size, bench configuration --
+@pytest.fixture(scope="module")
+def w100():
+    return chgen.generate(1, 101, seed=1, mode="spread")
+
+
+def test_full_size_w100_bench_config(h, w100):
+    """BASELINE configs[1]/[2] size (W=100, 30M order_line rows), launched exactly as bench.py
+    does (same engine entry points, default CH params), compared element by element."""
+    e = h.h2tap_open(0)
+    try:
+        h.h2tap_load_snapshot(e, h.hot_path_tables(w100), 1)
+        L = Loader(h, e)
+        assert_q6(L.q(6), oracle.q6(w100, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))
+        assert_q1(L.q(1), oracle.q1(w100, Q1_CUTOFF))
+        got = L.q(18, flags=h.H2TAP_QUERY_PROFILE)
+        assert_q18(got, oracle.q18(w100, Q18_HAVING))
+    finally:
+        h.h2tap_close(e)
