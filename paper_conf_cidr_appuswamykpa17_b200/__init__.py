@@ -38,6 +38,7 @@ H2TAP_FULL_RELOAD = 1
 H2TAP_LOAD_ASYNC = 1
 H2TAP_RESULT_DEVICE = 1
 H2TAP_QUERY_PROFILE = 2
+H2TAP_QUERY_HASH_JOIN = 4
 
 _DT = {H2TAP_I32: np.int32, H2TAP_I64: np.int64, H2TAP_F64: np.float64}
 
@@ -78,7 +79,7 @@ class h2tap_result(C.Structure):
                 ("nulls", C.POINTER(C.POINTER(C.c_uint8))), ("rows_scanned", C.c_uint64),
                 ("device_ms", C.c_double), ("e2e_ms", C.c_double), ("nkernels", C.c_uint32),
                 ("kernel_names", C.POINTER(C.c_char_p)), ("kernel_ms", C.POINTER(C.c_double)),
-                ("kernel_launches", C.c_uint64)]
+                ("kernel_launches", C.c_uint64), ("plan_flags", C.c_uint32)]
 
 
 _P = C.c_void_p
@@ -244,6 +245,7 @@ class Result:
             if bool(r.nulls[i]):
                 self.nulls[name] = np.ctypeslib.as_array(r.nulls[i], (self.nrows,)).copy()
         self.kernel_launches = r.kernel_launches
+        self.plan_flags = r.plan_flags
         self.kernels = [(r.kernel_names[i].decode(), r.kernel_ms[i]) for i in range(r.nkernels)]
 
     def to_numpy(self) -> dict:

@@ -193,11 +193,15 @@ struct ResultImpl : h2tap_result {
 };
 
 // =========================================================== snapshot ===
+constexpr int kStatCols = 3;  // min/max kept for the (w, d, id) key columns 0..2 of each table
 struct View {  // immutable snapshot at one epoch (the paper's shallow-copied top container)
     uint64_t epoch = 0;
     uint64_t n[kTables] = {};
     void *col[kTables][kMaxCols] = {};
     DevBufP keep[kTables][kMaxCols];
+    // column statistics of the visible rows (zone map): valid once the view is published
+    int smin[kTables][kStatCols], smax[kTables][kStatCols];
+    bool has_stats[kTables] = {};
 };
 using ViewP = std::shared_ptr<const View>;
 
@@ -214,8 +218,11 @@ struct TableState {
 
 struct Pending {
     uint64_t epoch;
-    ViewP view;
+    std::shared_ptr<View> view;   // becomes visible (const) at publish
     cudaEvent_t done;
+    bool loaded[kTables], full[kTables];
+    int *stats_host;              // pinned [kTables][kStatCols][2] delta min/max
+    std::pair<void *, size_t> stats_block;
 };
 
 struct Staging {  // pinned ring for pageable host buffers
@@ -285,7 +292,8 @@ struct h2tap_engine {
     std::deque<Pending> pending;
     Staging staging;
 
-    Arena arena;
+    Arena arena;       // query scratch (compute stream)
+    Arena load_arena;  // refresh scratch (copy stream)
     Prof prof;
     std::shared_ptr<BlockPool> host_pool, dev_pool;
     long long *small_host = nullptr;  // pinned scratch for tiny D2H reads
@@ -303,11 +311,30 @@ void publish_ready(h2tap_engine *e, bool wait) {
             if (q == cudaErrorNotReady) break;
             if (q != cudaSuccess) CK(q);
         }
+        {  // statistics: delta of this refresh merged onto the previous epoch's (R17)
+            View &v = *p.view;
+            const View *prev = e->published.get();
+            for (int t = 1; t < kTables; ++t) {
+                const bool carry = !p.full[t] && prev && prev->has_stats[t];
+                for (int c = 0; c < kStatCols; ++c) {
+                    int mn = INT32_MAX, mx = INT32_MIN;
+                    if (carry) { mn = prev->smin[t][c]; mx = prev->smax[t][c]; }
+                    if (p.loaded[t]) {
+                        mn = std::min(mn, p.stats_host[(t * kStatCols + c) * 2]);
+                        mx = std::max(mx, p.stats_host[(t * kStatCols + c) * 2 + 1]);
+                    }
+                    v.smin[t][c] = mn;
+                    v.smax[t][c] = mx;
+                }
+                v.has_stats[t] = p.loaded[t] || carry;
+            }
+        }
         {
             std::lock_guard<std::mutex> gv(e->view_mu);
             e->published = p.view;
         }
         cudaEventDestroy(p.done);
+        e->host_pool->put(p.stats_block.first, p.stats_block.second);
         e->pending.pop_front();
     }
 }
@@ -398,6 +425,12 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
     if (e->accepted) *v = *e->accepted;
     v->epoch = epoch;
     bool must_wait = false;
+    Pending pend{};
+    pend.epoch = epoch;
+    pend.stats_block = e->host_pool->get(sizeof(int) * kTables * kStatCols * 2);
+    pend.stats_host = static_cast<int *>(pend.stats_block.first);
+    int *stats_dev = static_cast<int *>(e->load_arena.get("load.stats", sizeof(int) * kTables * kStatCols * 2));
+    launch_stats_init(stats_dev, kTables * kStatCols, e->copy);
     for (uint32_t i = 0; i < ntables; ++i) {
         const h2tap_table &t = tables[i];
         TableState &ts = e->tables[t.table_id];
@@ -451,16 +484,28 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         }
         ts.loaded = t.row_count;
         v->n[t.table_id] = t.row_count;
+        pend.loaded[t.table_id] = true;
+        pend.full[t.table_id] = full;
+        // zone map of the appended rows' key columns, on the copy stream after their H2D
+        if (t.table_id != H2TAP_T_ITEM)
+            for (int c = 0; c < kStatCols; ++c)
+                if (v->col[t.table_id][c])
+                    launch_minmax_i32(static_cast<const int32_t *>(v->col[t.table_id][c]) + t.first_row,
+                                      t.row_count - t.first_row,
+                                      stats_dev + (t.table_id * kStatCols + c) * 2, e->num_sms, e->copy);
     }
-    cudaEvent_t done;
-    CK(cudaEventCreateWithFlags(&done, cudaEventDisableTiming));
-    CK(cudaEventRecord(done, e->copy));
+    CK(cudaGetLastError());
+    CK(cudaMemcpyAsync(pend.stats_host, stats_dev, sizeof(int) * kTables * kStatCols * 2,
+                       cudaMemcpyDeviceToHost, e->copy));
+    CK(cudaEventCreateWithFlags(&pend.done, cudaEventDisableTiming));
+    CK(cudaEventRecord(pend.done, e->copy));
+    pend.view = v;
     e->accepted = v;
     e->last_epoch = epoch;
     e->any_epoch = true;
     {
         std::lock_guard<std::mutex> gp(e->pend_mu);
-        e->pending.push_back(Pending{epoch, v, done});
+        e->pending.push_back(pend);
     }
     if (must_wait || !(flags & H2TAP_LOAD_ASYNC)) publish_ready(e, true);
     return H2TAP_OK;
@@ -636,24 +681,54 @@ uint64_t pow2_at_least(uint64_t x) {
     return c;
 }
 
-void run_q18(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
+// Planner for a join index on (w, d, id) = columns 0..2 of `table`: a perfect
+// hash over the key box of the build side when the box holds <= 4 slots per row, else an
+// open-addressing hash table. Statistics come from the published snapshot (zone maps).
+JoinIndex plan_index(h2tap_engine *e, const View &v, int table, bool force_hash, const char *name) {
+    JoinIndex j{};
+    const uint64_t n = v.n[table];
+    if (!force_hash && n && v.has_stats[table]) {
+        const long long nw = (long long)v.smax[table][0] - v.smin[table][0] + 1;
+        const long long nd = (long long)v.smax[table][1] - v.smin[table][1] + 1;
+        const long long nk = (long long)v.smax[table][2] - v.smin[table][2] + 1;
+        if (nw > 0 && nd > 0 && nk > 0) {
+            const double range = (double)nw * (double)nd * (double)nk;
+            if (range <= 4.0 * (double)n + 4096.0 && range < 4.0e9) {
+                j.dense = 1;
+                j.w0 = v.smin[table][0]; j.d0 = v.smin[table][1]; j.k0 = v.smin[table][2];
+                j.nw = (unsigned)nw; j.nd = (unsigned)nd; j.nk = (unsigned)nk;
+                j.range = (unsigned long long)nw * (unsigned long long)nd * (unsigned long long)nk;
+                j.slots = static_cast<unsigned int *>(
+                    e->arena.get(std::string(name) + ".dense", 4 * (j.range + 4)));
+                return j;
+            }
+        }
+    }
+    const uint64_t cap = pow2_at_least(2 * n);
+    j.dense = 0;
+    j.mask = cap - 1;
+    j.ht = static_cast<HtSlot *>(e->arena.get(std::string(name) + ".ht", sizeof(HtSlot) * cap));
+    return j;
+}
+
+void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, ResultImpl *r) {
     const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
     need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}, "Q18");
     need_cols(v, O, {H2TAP_O_W_ID, H2TAP_O_D_ID, H2TAP_O_ID, H2TAP_O_C_ID, H2TAP_O_OL_CNT, H2TAP_O_ENTRY_D}, "Q18");
     need_cols(v, C, {H2TAP_C_W_ID, H2TAP_C_D_ID, H2TAP_C_ID, H2TAP_C_LAST}, "Q18");
     const uint64_t n_ol = v.n[OL], n_o = v.n[O], n_c = v.n[C];
+    const bool force_hash = flags & H2TAP_QUERY_HASH_JOIN;
     Q18Scratch s;
-    s.cap_o = pow2_at_least(2 * n_o);
-    s.cap_c = pow2_at_least(2 * n_c);
-    s.ht_o = static_cast<HtSlot *>(e->arena.get("q18.ht_o", sizeof(HtSlot) * s.cap_o));
-    s.ht_c = static_cast<HtSlot *>(e->arena.get("q18.ht_c", sizeof(HtSlot) * s.cap_c));
+    s.jo = plan_index(e, v, O, force_hash, "q18.jo");
+    s.jc = plan_index(e, v, C, force_hash, "q18.jc");
     s.acc = static_cast<Q18Acc *>(e->arena.get("q18.acc", sizeof(Q18Acc) * std::max<uint64_t>(n_o, 1)));
     s.err = static_cast<unsigned int *>(e->arena.get("q18.err", 64));
     s.nout = static_cast<unsigned long long *>(e->arena.get("q18.nout", 64));
     s.stats = static_cast<Q18Stats *>(e->arena.get("q18.stats", sizeof(Q18Stats)));
-    s.un = carve_cols(e->arena, "q18.un.", n_o);
+    s.rows = static_cast<Q18Row *>(e->arena.get("q18.rows", sizeof(Q18Row) * std::max<uint64_t>(n_o, 1)));
+    r->plan_flags = (s.jo.dense ? 1u : 0u) | (s.jc.dense ? 2u : 0u);
 
-    e->prof.run("q18_init", [&] { launch_q18_init(s, n_o, e->compute); });
+    e->prof.run("q18_init", [&] { launch_q18_init(s, n_o, e->num_sms, e->compute); });
     e->prof.run("q18_build", [&] {
         launch_q18_build(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
                          colp<int32_t>(v, O, H2TAP_O_ID), n_o, colp<int32_t>(v, C, H2TAP_C_W_ID),
@@ -675,7 +750,7 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
     });
     CK(cudaGetLastError());
     // small D2H: err, nout, stats
-    struct Small { unsigned long long nout; unsigned int err, pad; Q18Stats st; };
+    struct Small { unsigned long long nout; unsigned int err, tie; Q18Stats st; };
     static_assert(sizeof(Small) <= 256, "small");
     Small *sm = reinterpret_cast<Small *>(e->small_host);
     CK(cudaMemcpyAsync(&sm->nout, s.nout, 8, cudaMemcpyDeviceToHost, e->compute));
@@ -698,7 +773,7 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
     if (err & kErrDomain) raise(H2TAP_EPLAN, "Q18: join key outside the supported domain");
     if (err_any) raise(H2TAP_EPLAN, "Q18: failed on another rank");
 
-    Q18Cols src = s.un;
+    const Q18Row *rows = s.rows;
     if (e->world > 1) {  // a7: groups are warehouse-local; gather result rows to rank 0
         auto *cnt_dev = static_cast<unsigned long long *>(e->arena.get("q18.allcnt", 8ull * e->world));
         NK(ncclAllGather(s.nout, cnt_dev, 1, ncclUint64, e->comm, e->compute));
@@ -707,27 +782,22 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
         sync_compute(e);
         uint64_t total = 0;
         for (auto c : cnts) total += c;
-        if (e->rank == 0) src = carve_cols(e->arena, "q18.all.", total);
+        Q18Row *all = e->rank == 0 ? static_cast<Q18Row *>(e->arena.get("q18.allrows", sizeof(Q18Row) * std::max<uint64_t>(total, 1)))
+                                   : nullptr;
         e->prof.run("q18_gather", [&] {
             NK(ncclGroupStart());
             uint64_t off = 0;
             for (int k = 0; k < e->world; ++k) {
-                const uint64_t c = cnts[k];
-                if (!c) continue;
-                auto xfer = [&](void *dst_base, const void *src_base, size_t es) {
+                const size_t bytes = cnts[k] * sizeof(Q18Row);
+                if (bytes) {
                     if (e->rank == 0 && k == 0)
-                        CK(cudaMemcpyAsync(static_cast<char *>(dst_base) + off * es, src_base, c * es,
-                                           cudaMemcpyDeviceToDevice, e->compute));
+                        CK(cudaMemcpyAsync(all, s.rows, bytes, cudaMemcpyDeviceToDevice, e->compute));
                     else if (e->rank == 0)
-                        NK(ncclRecv(static_cast<char *>(dst_base) + off * es, c * es, ncclUint8, k, e->comm, e->compute));
+                        NK(ncclRecv(all + off, bytes, ncclUint8, k, e->comm, e->compute));
                     else if (e->rank == k)
-                        NK(ncclSend(src_base, c * es, ncclUint8, 0, e->comm, e->compute));
-                };
-                xfer(src.c_last, s.un.c_last, 4); xfer(src.c_id, s.un.c_id, 4);
-                xfer(src.o_id, s.un.o_id, 4); xfer(src.o_ol_cnt, s.un.o_ol_cnt, 4);
-                xfer(src.o_w_id, s.un.o_w_id, 4); xfer(src.o_d_id, s.un.o_d_id, 4);
-                xfer(src.o_entry_d, s.un.o_entry_d, 8); xfer(src.amount_sum, s.un.amount_sum, 8);
-                off += c;
+                        NK(ncclSend(s.rows, bytes, ncclUint8, 0, e->comm, e->compute));
+                }
+                off += cnts[k];
             }
             NK(ncclGroupEnd());
         });
@@ -741,83 +811,119 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
             return;
         }
         nout = total;
-        // stats over the gathered rows
+        rows = all;
         Q18Stats init;
         init.amt_min = INT64_MAX; init.amt_max = INT64_MIN; init.ent_min = INT64_MAX; init.ent_max = INT64_MIN;
         init.w_min = INT32_MAX; init.w_max = INT32_MIN; init.d_min = INT32_MAX; init.d_max = INT32_MIN;
         init.o_min = INT32_MAX; init.o_max = INT32_MIN; init.pad0 = init.pad1 = 0;
         sm->st = init;
         CK(cudaMemcpyAsync(s.stats, &sm->st, sizeof(Q18Stats), cudaMemcpyHostToDevice, e->compute));
-        launch_q18_stats(src, nout, s.stats, e->num_sms, e->compute);
+        launch_q18_stats(rows, nout, s.stats, e->num_sms, e->compute);
         CK(cudaMemcpyAsync(&sm->st, s.stats, sizeof(Q18Stats), cudaMemcpyDeviceToHost, e->compute));
         sync_compute(e);
         st = sm->st;
     }
 
-    // a8: ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id — LSD radix sort
+    // a8: ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id — radix sort of row ids
+    Q18SortSpec sp{};
+    SortPairs sp2{};
     const unsigned int *perm = nullptr;
+    unsigned int *tie_dev = static_cast<unsigned int *>(e->arena.get("q18.tie", 64));
+    bool tiefix = false;
     if (nout > 1) {
-        Q18SortSpec sp;
         sp.amt_max = st.amt_max;
         sp.ent_min = st.ent_min;
         sp.w_min = st.w_min; sp.d_min = st.d_min; sp.o_min = st.o_min;
         sp.nd = (long long)st.d_max - st.d_min + 1;
         sp.no = (long long)st.o_max - st.o_min + 1;
         const unsigned long long nw = (unsigned long long)((long long)st.w_max - st.w_min + 1);
-        sp.bits[0] = bitwidth(nw * (unsigned long long)sp.nd * (unsigned long long)sp.no - 1);
-        sp.bits[1] = bitwidth((unsigned long long)st.ent_max - (unsigned long long)st.ent_min);
-        sp.bits[2] = bitwidth((unsigned long long)st.amt_max - (unsigned long long)st.amt_min);
-        SortScratch ss;
-        ss.max_n = nout;
-        for (int f = 0; f < 3; ++f)
-            ss.key[f] = static_cast<unsigned long long *>(e->arena.get("q18.sk" + std::to_string(f), 8 * nout));
-        ss.idx_a = static_cast<unsigned int *>(e->arena.get("q18.idxa", 4 * nout));
-        ss.idx_b = static_cast<unsigned int *>(e->arena.get("q18.idxb", 4 * nout));
-        const uint64_t tiles = (nout + 8191) / 8192;
-        ss.counts = static_cast<unsigned int *>(e->arena.get("q18.counts", 4ull * 256 * tiles));
-        e->prof.run("q18_sort_keys", [&] { launch_q18_sort_keys(src, nout, sp, ss, e->num_sms, e->compute); });
-        e->prof.run("q18_radix_sort", [&] { perm = radix_sort_fields(nout, sp.bits, ss, e->compute, e->num_sms); });
+        sp.bits_a = bitwidth((unsigned long long)st.amt_max - (unsigned long long)st.amt_min);
+        sp.bits_e = bitwidth((unsigned long long)st.ent_max - (unsigned long long)st.ent_min);
+        sp.bits_r = bitwidth(nw * (unsigned long long)sp.nd * (unsigned long long)sp.no - 1);
+        const int B = sp.bits_a + sp.bits_e + sp.bits_r;
+        sp.prefix_bits = B <= 64 ? B : 48;
+        tiefix = B > sp.prefix_bits;
+        for (int b = 0; b < 2; ++b) {
+            sp2.k[b] = static_cast<unsigned long long *>(e->arena.get("q18.sk" + std::to_string(b), 8 * nout));
+            sp2.v[b] = static_cast<unsigned int *>(e->arena.get("q18.sv" + std::to_string(b), 4 * nout));
+        }
+        sp2.counts = static_cast<unsigned int *>(e->arena.get("q18.counts", 4ull * 256 * sort_tiles(nout)));
+        sp2.totals = static_cast<unsigned int *>(e->arena.get("q18.totals", 4 * 256));
+        e->prof.run("q18_sort_keys", [&] { launch_q18_sort_keys(rows, nout, sp, sp2, e->num_sms, e->compute); });
+        int cur = 0;
+        e->prof.run("q18_radix_sort", [&] { cur = radix_sort_pairs(nout, sp.prefix_bits, sp2, e->num_sms, e->compute); });
+        perm = sp2.v[cur];
+        if (tiefix) {
+            CK(cudaMemsetAsync(tie_dev, 0, 4, e->compute));
+            e->prof.run("q18_tiefix", [&] {
+                launch_q18_tiefix(rows, sp2.k[cur], sp2.v[cur], nout, tie_dev, e->num_sms, e->compute);
+            });
+        }
     }
     r->nrows = nout;
     Q18Cols dst;
-    if (r->on_device) {
-        dst.c_last = static_cast<int32_t *>(result_block(r, 4 * nout));
-        dst.c_id = static_cast<int32_t *>(result_block(r, 4 * nout));
-        dst.o_id = static_cast<int32_t *>(result_block(r, 4 * nout));
-        dst.o_entry_d = static_cast<int64_t *>(result_block(r, 8 * nout));
-        dst.o_ol_cnt = static_cast<int32_t *>(result_block(r, 4 * nout));
-        dst.amount_sum = static_cast<int64_t *>(result_block(r, 8 * nout));
-        dst.o_w_id = static_cast<int32_t *>(result_block(r, 4 * nout));
-        dst.o_d_id = static_cast<int32_t *>(result_block(r, 4 * nout));
-        e->prof.run("q18_permute", [&] { if (nout) launch_q18_permute(src, perm, nout, dst, e->num_sms, e->compute); });
-    } else {
-        Q18Cols sorted = carve_cols(e->arena, "q18.sorted.", nout);
-        e->prof.run("q18_permute", [&] { if (nout) launch_q18_permute(src, perm, nout, sorted, e->num_sms, e->compute); });
-        auto d2h = [&](const void *src_p, size_t es) {
-            void *h = result_block(r, nout * es);
-            if (nout) CK(cudaMemcpyAsync(h, src_p, nout * es, cudaMemcpyDeviceToHost, e->compute));
-            return h;
-        };
-        dst.c_last = static_cast<int32_t *>(d2h(sorted.c_last, 4));
-        dst.c_id = static_cast<int32_t *>(d2h(sorted.c_id, 4));
-        dst.o_id = static_cast<int32_t *>(d2h(sorted.o_id, 4));
-        dst.o_entry_d = static_cast<int64_t *>(d2h(sorted.o_entry_d, 8));
-        dst.o_ol_cnt = static_cast<int32_t *>(d2h(sorted.o_ol_cnt, 4));
-        dst.amount_sum = static_cast<int64_t *>(d2h(sorted.amount_sum, 8));
-        dst.o_w_id = static_cast<int32_t *>(d2h(sorted.o_w_id, 4));
-        dst.o_d_id = static_cast<int32_t *>(d2h(sorted.o_d_id, 4));
+    auto alloc_dst = [&](bool device) {
+        auto blk = [&](size_t es) { return result_block(r, es * nout); };
+        if (device) {
+            dst.c_last = static_cast<int32_t *>(blk(4)); dst.c_id = static_cast<int32_t *>(blk(4));
+            dst.o_id = static_cast<int32_t *>(blk(4)); dst.o_entry_d = static_cast<int64_t *>(blk(8));
+            dst.o_ol_cnt = static_cast<int32_t *>(blk(4)); dst.amount_sum = static_cast<int64_t *>(blk(8));
+            dst.o_w_id = static_cast<int32_t *>(blk(4)); dst.o_d_id = static_cast<int32_t *>(blk(4));
+        }
+    };
+    Q18Cols host_dst{};
+    if (r->on_device) alloc_dst(true);
+    else {
+        dst = carve_cols(e->arena, "q18.sorted.", nout);
+        host_dst.c_last = static_cast<int32_t *>(result_block(r, 4 * nout));
+        host_dst.c_id = static_cast<int32_t *>(result_block(r, 4 * nout));
+        host_dst.o_id = static_cast<int32_t *>(result_block(r, 4 * nout));
+        host_dst.o_entry_d = static_cast<int64_t *>(result_block(r, 8 * nout));
+        host_dst.o_ol_cnt = static_cast<int32_t *>(result_block(r, 4 * nout));
+        host_dst.amount_sum = static_cast<int64_t *>(result_block(r, 8 * nout));
+        host_dst.o_w_id = static_cast<int32_t *>(result_block(r, 4 * nout));
+        host_dst.o_d_id = static_cast<int32_t *>(result_block(r, 4 * nout));
     }
-    CK(cudaGetLastError());
-    CK(cudaEventRecord(e->q_end, e->compute));
-    sync_compute(e);
-    add_col(r, "c_last", H2TAP_I32, dst.c_last);
-    add_col(r, "c_id", H2TAP_I32, dst.c_id);
-    add_col(r, "o_id", H2TAP_I32, dst.o_id);
-    add_col(r, "o_entry_d", H2TAP_I64, dst.o_entry_d);
-    add_col(r, "o_ol_cnt", H2TAP_I32, dst.o_ol_cnt);
-    add_col(r, "amount_sum", H2TAP_I64, dst.amount_sum);
-    add_col(r, "o_w_id", H2TAP_I32, dst.o_w_id);
-    add_col(r, "o_d_id", H2TAP_I32, dst.o_d_id);
+    auto emit = [&]() {
+        e->prof.run("q18_permute", [&] { if (nout) launch_q18_permute(rows, perm, nout, dst, e->num_sms, e->compute); });
+        if (!r->on_device && nout) {
+            auto d2h = [&](void *h, const void *d, size_t es) {
+                CK(cudaMemcpyAsync(h, d, nout * es, cudaMemcpyDeviceToHost, e->compute));
+            };
+            d2h(host_dst.c_last, dst.c_last, 4); d2h(host_dst.c_id, dst.c_id, 4);
+            d2h(host_dst.o_id, dst.o_id, 4); d2h(host_dst.o_entry_d, dst.o_entry_d, 8);
+            d2h(host_dst.o_ol_cnt, dst.o_ol_cnt, 4); d2h(host_dst.amount_sum, dst.amount_sum, 8);
+            d2h(host_dst.o_w_id, dst.o_w_id, 4); d2h(host_dst.o_d_id, dst.o_d_id, 4);
+        }
+        if (tiefix) CK(cudaMemcpyAsync(&sm->tie, tie_dev, 4, cudaMemcpyDeviceToHost, e->compute));
+        CK(cudaGetLastError());
+        CK(cudaEventRecord(e->q_end, e->compute));
+        sync_compute(e);
+    };
+    emit();
+    if (tiefix && sm->tie) {
+        // a run of > 32 equal prefixes: redo exactly, one stable LSD sort per field (r, e, a)
+        SortPairs w = sp2;
+        launch_iota(w.v[0], nout, e->num_sms, e->compute);
+        const int fb[3] = {sp.bits_r, sp.bits_e, sp.bits_a};
+        for (int f = 0; f < 3; ++f) {
+            launch_q18_field_keys(rows, w.v[0], nout, f, sp, w.k[0], e->num_sms, e->compute);
+            const int cur = radix_sort_pairs(nout, fb[f], w, e->num_sms, e->compute);
+            if (cur) { std::swap(w.k[0], w.k[1]); std::swap(w.v[0], w.v[1]); }
+        }
+        perm = w.v[0];
+        tiefix = false;
+        emit();
+    }
+    const Q18Cols &out = r->on_device ? dst : host_dst;
+    add_col(r, "c_last", H2TAP_I32, out.c_last);
+    add_col(r, "c_id", H2TAP_I32, out.c_id);
+    add_col(r, "o_id", H2TAP_I32, out.o_id);
+    add_col(r, "o_entry_d", H2TAP_I64, out.o_entry_d);
+    add_col(r, "o_ol_cnt", H2TAP_I32, out.o_ol_cnt);
+    add_col(r, "amount_sum", H2TAP_I64, out.amount_sum);
+    add_col(r, "o_w_id", H2TAP_I32, out.o_w_id);
+    add_col(r, "o_d_id", H2TAP_I32, out.o_d_id);
 }
 
 // CH-benCHmark constants as int64 µs UTC / cents (R4, R6).
@@ -860,7 +966,7 @@ h2tap_status query_impl(h2tap_engine *e, uint32_t plan, const int64_t *params, u
     switch (plan) {
         case H2TAP_Q1: run_q1(e, *v, p, r.get()); break;
         case H2TAP_Q6: run_q6(e, *v, p, r.get()); break;
-        case H2TAP_Q18: run_q18(e, *v, p, r.get()); break;
+        case H2TAP_Q18: run_q18(e, *v, p, flags, r.get()); break;
     }
     float ms = 0;
     CK(cudaEventElapsedTime(&ms, e->q_begin, e->q_end));
@@ -924,6 +1030,7 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         CK(cudaEventCreate(&e->q_end));
         CK(cudaMallocHost(&e->small_host, 256));
         e->arena.device = e->device;
+        e->load_arena.device = e->device;
         e->host_pool = std::make_shared<BlockPool>(true, e->device);
         e->dev_pool = std::make_shared<BlockPool>(false, e->device);
         if (e->world > 1) {
@@ -981,7 +1088,10 @@ void h2tap_close(h2tap_engine *e) {
     cudaStreamSynchronize(e->compute);
     cudaStreamSynchronize(e->copy);
     if (e->comm) ncclCommDestroy(e->comm);
-    for (auto &p : e->pending) cudaEventDestroy(p.done);
+    for (auto &p : e->pending) {
+        cudaEventDestroy(p.done);
+        e->host_pool->put(p.stats_block.first, p.stats_block.second);
+    }
     for (int k = 0; k < Staging::kSlots; ++k) {
         if (e->staging.buf[k]) cudaFreeHost(e->staging.buf[k]);
         if (e->staging.ev[k]) cudaEventDestroy(e->staging.ev[k]);
@@ -994,6 +1104,7 @@ void h2tap_close(h2tap_engine *e) {
     e->accepted.reset();
     for (auto &t : e->tables) for (auto &c : t.col) { c.cur.reset(); c.spare.reset(); }
     e->arena.bufs.clear();
+    e->load_arena.bufs.clear();
     cudaStreamDestroy(e->compute);
     cudaStreamDestroy(e->copy);
     delete e;

@@ -1,13 +1,16 @@
-// join_kernels.cu — K3 hash build, K4 probe + group-join aggregation, K5 HAVING + compaction +
-// customer probe + gather, for CH Q18 (customer ⋈ orders ⋈ order_line, GROUP BY, HAVING) on sm_100a.
+// join_kernels.cu — K3 join-index build, K4 probe + group-join aggregation, K5 HAVING +
+// compaction + customer probe + gather, for CH Q18 (customer ⋈ orders ⋈ order_line, GROUP BY,
+// HAVING) on sm_100a.
 //
 // The paper gives no join algorithm (hash joins on accelerators appear only as related work,
 // PAPER.md L1224-1227); its runtime hands kernels the snapshot's column pointers (L568-570).
-// Design: open-addressing hash tables with 16-byte slots {packed key, row},
-// linear probing, capacity a power of two >= 2n, insert by 64-bit atomicCAS. Q18's GROUP BY
-// key (o_id, o_w_id, o_d_id, c_id, c_last, o_entry_d, o_ol_cnt) is functionally determined by
-// the orders primary key once orders and customer PKs are unique (checked: EDUPKEY), so the
-// group-by collapses onto the orders row: acc[orders row] += (amount, 1).
+// Design: a join index per build side maps the primary key (w, d, id) to a row.
+// It is a perfect hash (slot = dense rank of the key in the build side's [min, max] box, from
+// the snapshot's column statistics) when that box is small, else an open-addressing hash table
+// (16-byte slots, linear probing, capacity pow2 >= 2n, insert by 64-bit atomicCAS). Q18's
+// GROUP BY key (o_id, o_w_id, o_d_id, c_id, c_last, o_entry_d, o_ol_cnt) is functionally
+// determined by the orders row once the orders and customer PKs are unique (checked:
+// EDUPKEY), so the group-by collapses onto the orders row: acc[orders row] += (amount, 1).
 #include <cstdint>
 #include <cuda_runtime.h>
 
@@ -17,51 +20,89 @@ namespace h2tap {
 namespace {
 
 constexpr unsigned kFull = 0xffffffffu;
-constexpr unsigned int kNone = 0xffffffffu;
 
 __device__ __forceinline__ unsigned long long fmix64(unsigned long long k) {
     k ^= k >> 33; k *= 0xff51afd7ed558ccdull; k ^= k >> 33; k *= 0xc4ceb9fe1a85ec53ull; k ^= k >> 33;
     return k;
 }
 
-// (w, d, id) -> 64-bit key, order-preserving on the supported domain (R16).
+// (w, d, id) -> 64-bit key, injective on the supported domain (R16).
 __device__ __forceinline__ bool pack_key(int w, int d, int id, unsigned long long &k) {
     k = ((unsigned long long)(unsigned)w << 40) | ((unsigned long long)(unsigned)d << 32) |
         (unsigned long long)(unsigned)id;
     return ((unsigned)w < (1u << 23)) & ((unsigned)d < 256u) & (id >= 0);
 }
 
-__device__ __forceinline__ void ht_insert(HtSlot *ht, unsigned long long mask, unsigned long long key,
-                                          unsigned int row, unsigned int *err, unsigned int dupbit) {
-    unsigned long long h = fmix64(key) & mask;
+// Dense slot of (w, d, id) in the index's box, or false when outside it.
+__device__ __forceinline__ bool dense_slot(const JoinIndex &j, int w, int d, int id,
+                                          unsigned long long &slot) {
+    const unsigned dw = (unsigned)(w - j.w0), dd = (unsigned)(d - j.d0), dk = (unsigned)(id - j.k0);
+    slot = ((unsigned long long)dw * j.nd + dd) * j.nk + dk;
+    return (dw < j.nw) & (dd < j.nd) & (dk < j.nk);
+}
+
+// Insert; returns false on a key outside the supported domain. Duplicates set `dupbit`.
+__device__ __forceinline__ bool jx_insert(const JoinIndex &j, int w, int d, int id, unsigned int row,
+                                          unsigned int *err, unsigned int dupbit) {
+    if (j.dense) {
+        unsigned long long s;
+        if (!dense_slot(j, w, d, id, s)) return false;  // stats must cover every build row
+        if (atomicCAS(j.slots + s, kNoRow, row) != kNoRow) atomicOr(err, dupbit);
+        return true;
+    }
+    unsigned long long key;
+    if (!pack_key(w, d, id, key)) return false;
+    unsigned long long h = fmix64(key) & j.mask;
     while (true) {
-        const unsigned long long prev = atomicCAS(&ht[h].key, kEmpty, key);
-        if (prev == kEmpty) { ht[h].row = row; return; }
-        if (prev == key) { atomicOr(err, dupbit); return; }
-        h = (h + 1) & mask;
+        const unsigned long long prev = atomicCAS(&j.ht[h].key, kEmpty, key);
+        if (prev == kEmpty) { j.ht[h].row = row; return true; }
+        if (prev == key) { atomicOr(err, dupbit); return true; }
+        h = (h + 1) & j.mask;
     }
 }
 
-__device__ __forceinline__ unsigned int ht_probe(const HtSlot *ht, unsigned long long mask,
-                                                 unsigned long long key) {
-    unsigned long long h = fmix64(key) & mask;
-    while (true) {
-        const ulonglong2 s = __ldcg(reinterpret_cast<const ulonglong2 *>(ht + h));
-        if (s.x == key) return (unsigned int)s.y;
-        if (s.x == kEmpty) return kNone;
-        h = (h + 1) & mask;
+__device__ __forceinline__ unsigned int jx_lookup(const JoinIndex &j, int w, int d, int id) {
+    if (j.dense) {
+        unsigned long long s;
+        if (!dense_slot(j, w, d, id, s)) return kNoRow;  // outside the build box: no match
+        return __ldcg(j.slots + s);
     }
+    unsigned long long key;
+    if (!pack_key(w, d, id, key)) return kNoRow;  // no build key can lie outside the domain
+    unsigned long long h = fmix64(key) & j.mask;
+    while (true) {
+        const ulonglong2 s = __ldcg(reinterpret_cast<const ulonglong2 *>(j.ht + h));
+        if (s.x == key) return (unsigned int)s.y;
+        if (s.x == kEmpty) return kNoRow;
+        h = (h + 1) & j.mask;
+    }
+}
+
+unsigned grid_for(uint64_t work, int threads, int num_sms, int per_sm) {
+    uint64_t want = (work + threads - 1) / threads;
+    uint64_t cap = (uint64_t)num_sms * per_sm;
+    if (want > cap) want = cap;
+    return want ? (unsigned)want : 1u;
 }
 
 // ------------------------------------------------------------------- init --
+// Empties both join indexes, zeroes the group accumulators and the counters: one launch.
+__host__ __device__ __forceinline__ uint64_t jx_words(const JoinIndex &j) {  // 16-byte units
+    return j.dense ? (j.range + 3) / 4 : j.mask + 1;
+}
+__device__ __forceinline__ void jx_clear(const JoinIndex &j, uint64_t i) {
+    if (j.dense) reinterpret_cast<uint4 *>(j.slots)[i] = make_uint4(kNoRow, kNoRow, kNoRow, kNoRow);
+    else reinterpret_cast<ulonglong2 *>(j.ht)[i] = make_ulonglong2(kEmpty, 0ull);
+}
+
 __global__ void q18_init_kernel(Q18Scratch s, uint64_t n_orders) {
-    const uint64_t total = s.cap_o + s.cap_c + n_orders;
+    const uint64_t a = jx_words(s.jo), b = jx_words(s.jc);
+    const uint64_t total = a + b + n_orders;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    const ulonglong2 empty = make_ulonglong2(kEmpty, 0ull), zero = make_ulonglong2(0ull, 0ull);
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < total; i += stride) {
-        if (i < s.cap_o) reinterpret_cast<ulonglong2 *>(s.ht_o)[i] = empty;
-        else if (i < s.cap_o + s.cap_c) reinterpret_cast<ulonglong2 *>(s.ht_c)[i - s.cap_o] = empty;
-        else reinterpret_cast<ulonglong2 *>(s.acc)[i - s.cap_o - s.cap_c] = zero;
+        if (i < a) jx_clear(s.jo, i);
+        else if (i < a + b) jx_clear(s.jc, i - a);
+        else reinterpret_cast<ulonglong2 *>(s.acc)[i - a - b] = make_ulonglong2(0ull, 0ull);
     }
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         *s.err = 0;
@@ -80,27 +121,25 @@ __global__ void q18_build_kernel(const int32_t *__restrict__ o_w, const int32_t 
                                  const int32_t *__restrict__ c_w, const int32_t *__restrict__ c_d,
                                  const int32_t *__restrict__ c_id, uint64_t n_c, Q18Scratch s) {
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    const unsigned long long mo = s.cap_o - 1, mc = s.cap_c - 1;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n_o + n_c; i += stride) {
-        unsigned long long k;
+        bool ok;
         if (i < n_o) {
-            if (!pack_key(o_w[i], o_d[i], o_id[i], k)) { atomicOr(s.err, kErrDomain); continue; }
-            ht_insert(s.ht_o, mo, k, (unsigned int)i, s.err, kErrDupOrders);
+            ok = jx_insert(s.jo, o_w[i], o_d[i], o_id[i], (unsigned int)i, s.err, kErrDupOrders);
         } else {
             const uint64_t j = i - n_o;
-            if (!pack_key(c_w[j], c_d[j], c_id[j], k)) { atomicOr(s.err, kErrDomain); continue; }
-            ht_insert(s.ht_c, mc, k, (unsigned int)j, s.err, kErrDupCustomer);
+            ok = jx_insert(s.jc, c_w[j], c_d[j], c_id[j], (unsigned int)j, s.err, kErrDupCustomer);
         }
+        if (!ok) atomicOr(s.err, kErrDomain);
     }
 }
 
 // ------------------------------------------------------- K4 probe + group-join --
 // One warp iteration covers 32 consecutive order_line rows (coalesced 4 B / 8 B loads).
 // Lines of one order are usually contiguous, so equal keys form runs: a segmented inclusive
-// scan (shuffles) sums each run, the run head probes the orders table once, and the run tail
+// scan (shuffles) sums each run, the run head probes the orders index once, and the run tail
 // issues the two atomics — ~3 runs per 32 rows instead of 32 probes and 64 atomics.
 constexpr int kProbeThreads = 256;
-constexpr int kProbeUnroll = 2;
+constexpr int kProbeUnroll = 4;
 
 __global__ void __launch_bounds__(kProbeThreads)
 q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ ol_d,
@@ -109,26 +148,29 @@ q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ o
     const int lane = threadIdx.x & 31;
     const uint64_t gwarp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
-    const unsigned long long mask = s.cap_o - 1;
     const unsigned le_mask = 0xffffffffu >> (31 - lane);  // lanes 0..lane
     for (uint64_t base = gwarp * 32 * kProbeUnroll; base < n; base += nwarps * 32 * kProbeUnroll) {
-        unsigned long long key[kProbeUnroll];
+        int w[kProbeUnroll], d[kProbeUnroll], o[kProbeUnroll];
         long long amt[kProbeUnroll];
+        bool valid[kProbeUnroll];
 #pragma unroll
         for (int u = 0; u < kProbeUnroll; ++u) {
             const uint64_t i = base + u * 32 + lane;
-            key[u] = kEmpty;  // invalid rows (tail / out of domain) never match
-            amt[u] = 0;
-            if (i < n) {
-                unsigned long long k;
-                if (pack_key(__ldcs(ol_w + i), __ldcs(ol_d + i), __ldcs(ol_o + i), k)) key[u] = k;
+            valid[u] = i < n;
+            if (valid[u]) {
+                w[u] = __ldcs(ol_w + i); d[u] = __ldcs(ol_d + i); o[u] = __ldcs(ol_o + i);
                 amt[u] = __ldcs(ol_amt + i);
+            } else {  // tail rows: never probe, never aggregate
+                w[u] = 0; d[u] = 0; o[u] = 0; amt[u] = 0;
             }
         }
 #pragma unroll
         for (int u = 0; u < kProbeUnroll; ++u) {
-            const unsigned long long prev = __shfl_up_sync(kFull, key[u], 1);
-            const bool head = lane == 0 || key[u] != prev;
+            const bool same = (__shfl_up_sync(kFull, w[u], 1) == w[u]) &
+                              (__shfl_up_sync(kFull, d[u], 1) == d[u]) &
+                              (__shfl_up_sync(kFull, o[u], 1) == o[u]) &
+                              (__shfl_up_sync(kFull, (int)valid[u], 1) == (int)valid[u]);
+            const bool head = lane == 0 || !same;
             const unsigned heads = __ballot_sync(kFull, head);
             const int leader = 31 - __clz(heads & le_mask);
             long long sum = amt[u];
@@ -138,10 +180,10 @@ q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ o
                 if (lane - off >= leader) sum += t;
             }
             const bool tail = lane == 31 || ((heads >> (lane + 1)) & 1u);
-            unsigned int row = kNone;
-            if (head && key[u] != kEmpty) row = ht_probe(s.ht_o, mask, key[u]);
+            unsigned int row = kNoRow;
+            if (head && valid[u]) row = jx_lookup(s.jo, w[u], d[u], o[u]);
             row = __shfl_sync(kFull, row, leader);
-            if (tail && row != kNone) {
+            if (tail && row != kNoRow) {
                 atomicAdd(reinterpret_cast<unsigned long long *>(&s.acc[row].sum),
                           (unsigned long long)sum);
                 atomicAdd(&s.acc[row].cnt, (unsigned int)(lane - leader + 1));
@@ -161,8 +203,6 @@ __device__ __forceinline__ long long wmax64(long long v) {
     for (int o = 16; o; o >>= 1) { long long t = __shfl_xor_sync(kFull, v, o); v = t > v ? t : v; }
     return v;
 }
-__device__ __forceinline__ int wmin32(int v) { return __reduce_min_sync(kFull, v); }
-__device__ __forceinline__ int wmax32(int v) { return __reduce_max_sync(kFull, v); }
 
 struct StatAcc {
     long long amin = INT64_MAX, amax = INT64_MIN, emin = INT64_MAX, emax = INT64_MIN;
@@ -176,8 +216,9 @@ struct StatAcc {
     }
     __device__ void flush(Q18Stats *st) {  // warp-reduce, lane 0 issues the atomics
         amin = wmin64(amin); amax = wmax64(amax); emin = wmin64(emin); emax = wmax64(emax);
-        wmin = wmin32(wmin); wmax = wmax32(wmax); dmin = wmin32(dmin); dmax = wmax32(dmax);
-        omin = wmin32(omin); omax = wmax32(omax);
+        wmin = __reduce_min_sync(kFull, wmin); wmax = __reduce_max_sync(kFull, wmax);
+        dmin = __reduce_min_sync(kFull, dmin); dmax = __reduce_max_sync(kFull, dmax);
+        omin = __reduce_min_sync(kFull, omin); omax = __reduce_max_sync(kFull, omax);
         if ((threadIdx.x & 31) == 0 && amin <= amax) {
             atomicMin(&st->amt_min, amin); atomicMax(&st->amt_max, amax);
             atomicMin(&st->ent_min, emin); atomicMax(&st->ent_max, emax);
@@ -196,12 +237,11 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
     const int lane = threadIdx.x & 31;
     const uint64_t gwarp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
-    const unsigned long long mc = s.cap_c - 1;
     StatAcc stat;
     for (uint64_t base = gwarp * 32; base < n; base += nwarps * 32) {
         const uint64_t r = base + lane;
         bool pass = false;
-        unsigned int crow = kNone;
+        unsigned int crow = kNoRow;
         long long sum = 0;
         int w = 0, d = 0, c = 0;
         if (r < n) {
@@ -211,9 +251,8 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
             // inner join: a group exists only with >= 1 order_line row; HAVING SUM > having
             if (cnt > 0 && sum > having) {
                 w = o_w[r]; d = o_d[r]; c = o_c[r];
-                unsigned long long k;
-                if (pack_key(w, d, c, k)) crow = ht_probe(s.ht_c, mc, k);  // c ⋈ o
-                pass = crow != kNone;
+                crow = jx_lookup(s.jc, w, d, c);  // customer ⋈ orders
+                pass = crow != kNoRow;
             }
         }
         const unsigned ball = __ballot_sync(kFull, pass);
@@ -223,49 +262,37 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
         basepos = __shfl_sync(kFull, basepos, 0);
         if (pass) {
             const uint64_t p = basepos + __popc(ball & ((1u << lane) - 1u));
-            const int oid = o_id[r];
-            const long long ent = o_ent[r];
-            s.un.c_last[p] = c_last[crow];
-            s.un.c_id[p] = c;
-            s.un.o_id[p] = oid;
-            s.un.o_entry_d[p] = ent;
-            s.un.o_ol_cnt[p] = o_cnt[r];
-            s.un.amount_sum[p] = sum;
-            s.un.o_w_id[p] = w;
-            s.un.o_d_id[p] = d;
-            stat.add(sum, ent, w, d, oid);
+            Q18Row row;
+            row.amount_sum = sum;
+            row.o_entry_d = o_ent[r];
+            row.c_last = c_last[crow];
+            row.c_id = c;
+            row.o_id = o_id[r];
+            row.o_ol_cnt = o_cnt[r];
+            row.o_w_id = w;
+            row.o_d_id = d;
+            s.rows[p] = row;
+            stat.add(sum, row.o_entry_d, w, d, row.o_id);
         }
     }
     stat.flush(s.stats);
 }
 
-__global__ void q18_stats_kernel(Q18Cols cols, uint64_t n, Q18Stats *st) {
+__global__ void q18_stats_kernel(const Q18Row *__restrict__ rows, uint64_t n, Q18Stats *st) {
     StatAcc stat;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride)
-        stat.add(cols.amount_sum[i], cols.o_entry_d[i], cols.o_w_id[i], cols.o_d_id[i], cols.o_id[i]);
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
+        const Q18Row r = rows[i];
+        stat.add(r.amount_sum, r.o_entry_d, r.o_w_id, r.o_d_id, r.o_id);
+    }
     stat.flush(st);
-}
-
-__global__ void fill_u64_kernel(unsigned long long *p, uint64_t n, unsigned long long v) {
-    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) p[i] = v;
-}
-
-unsigned grid_for(uint64_t work, int threads, int num_sms, int per_sm) {
-    uint64_t want = (work + threads - 1) / threads;
-    uint64_t cap = (uint64_t)num_sms * per_sm;
-    if (want > cap) want = cap;
-    return want ? (unsigned)want : 1u;
 }
 
 }  // namespace
 
-void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, cudaStream_t st) {
-    int dev = 0, sms = 148;
-    cudaGetDevice(&dev);
-    cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-    q18_init_kernel<<<grid_for(s.cap_o + s.cap_c + n_orders, 256, sms, 8), 256, 0, st>>>(s, n_orders);
+void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st) {
+    const uint64_t words = jx_words(s.jo) + jx_words(s.jc) + n_orders;
+    q18_init_kernel<<<grid_for(words, 256, num_sms, 8), 256, 0, st>>>(s, n_orders);
     count_launches(1);
 }
 
@@ -291,17 +318,12 @@ void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_
                        const Q18Scratch &s, int num_sms, cudaStream_t st) {
     q18_having_kernel<<<grid_for(n_o, kHavingThreads, num_sms, 8), kHavingThreads, 0, st>>>(
         o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o, c_last, having, s);
-        count_launches(1);
-}
-
-void launch_q18_stats(const Q18Cols &cols, uint64_t n, Q18Stats *stats, int num_sms,
-                      cudaStream_t st) {
-    q18_stats_kernel<<<grid_for(n, 256, num_sms, 4), 256, 0, st>>>(cols, n, stats);
     count_launches(1);
 }
 
-void launch_fill_u64(unsigned long long *p, uint64_t n, unsigned long long v, cudaStream_t st) {
-    fill_u64_kernel<<<grid_for(n, 256, 148, 8), 256, 0, st>>>(p, n, v);
+void launch_q18_stats(const Q18Row *rows, uint64_t n, Q18Stats *stats, int num_sms,
+                      cudaStream_t st) {
+    q18_stats_kernel<<<grid_for(n, 256, num_sms, 4), 256, 0, st>>>(rows, n, stats);
     count_launches(1);
 }
 

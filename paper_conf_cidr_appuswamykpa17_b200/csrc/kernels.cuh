@@ -50,27 +50,44 @@ void launch_q1_emit(const Q1Scratch &s, uint64_t ngroups, cudaStream_t st);  // 
 // ------------------------------------------------------------ Q18 (K3-K5) --
 struct HtSlot { unsigned long long key; unsigned int row; unsigned int pad; };  // 16 B
 constexpr unsigned long long kEmpty = ~0ull;
+constexpr unsigned int kNoRow = 0xffffffffu;
 struct Q18Acc { long long sum; unsigned int cnt; unsigned int pad; };          // 16 B
 enum : unsigned int { kErrDupOrders = 1u, kErrDupCustomer = 2u, kErrDomain = 4u };
 
+// Join index on a (w, d, id) primary key -> row. Two layouts, chosen per query by the planner
+// from the snapshot's column statistics:
+//  - dense: a perfect hash — slot = rank of (w, d, id) in the [min, max] box of the build side;
+//    used when that box holds <= 4 slots per row (TPC-C keys are dense);
+//  - hash: open addressing, 16-byte slots {packed key, row}, linear probing, cap = pow2 >= 2n.
+struct JoinIndex {
+    int dense;
+    HtSlot *ht; unsigned long long mask;             // hash
+    unsigned int *slots;                              // dense: [range] row or kNoRow
+    int w0, d0, k0;                                   // dense: box minimum
+    unsigned int nw, nd, nk;                          // dense: box extents
+    unsigned long long range;                         // dense: nw * nd * nk
+};
 struct Q18Stats {            // min/max of the sort fields over result rows (atomics)
     long long amt_min, amt_max, ent_min, ent_max;
     int w_min, w_max, d_min, d_max, o_min, o_max, pad0, pad1;
+};
+struct Q18Row {              // one result row before ORDER BY (AoS: one 40-byte gather later)
+    long long amount_sum, o_entry_d;
+    int c_last, c_id, o_id, o_ol_cnt, o_w_id, o_d_id;
 };
 struct Q18Cols {             // SoA result columns
     int32_t *c_last, *c_id, *o_id, *o_ol_cnt, *o_w_id, *o_d_id;
     int64_t *o_entry_d, *amount_sum;
 };
 struct Q18Scratch {
-    HtSlot *ht_o; uint64_t cap_o;
-    HtSlot *ht_c; uint64_t cap_c;
+    JoinIndex jo, jc;
     Q18Acc *acc;             // [n_orders]
     unsigned int *err;       // [1]
     unsigned long long *nout;// [1]
     Q18Stats *stats;         // [1]
-    Q18Cols un;              // unsorted result columns [n_orders]
+    Q18Row *rows;            // [n_orders] unsorted result rows
 };
-void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, cudaStream_t st);
+void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st);
 void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
                       const int32_t *c_w, const int32_t *c_d, const int32_t *c_id, uint64_t n_c,
                       const Q18Scratch &s, int num_sms, cudaStream_t st);
@@ -81,37 +98,53 @@ void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_
                        const int32_t *o_c, const int32_t *o_cnt, const int64_t *o_ent,
                        uint64_t n_o, const int32_t *c_last, int64_t having,
                        const Q18Scratch &s, int num_sms, cudaStream_t st);
-void launch_q18_stats(const Q18Cols &cols, uint64_t n, Q18Stats *stats, int num_sms,
+void launch_q18_stats(const Q18Row *rows, uint64_t n, Q18Stats *stats, int num_sms,
                       cudaStream_t st);  // recompute stats over gathered rows (multi-GPU)
 
 // ------------------------------------------------------------------ sort ---
-// Stable LSD radix sort of a permutation by up to three unsigned key fields (least significant
-// field first), 8-bit digits, only as many passes as each field's bit width needs.
-struct SortScratch {
-    unsigned long long *key[3];  // [n] per field
-    unsigned int *idx_a, *idx_b; // [n]
-    unsigned int *counts;        // [256 * max_tiles]
-    size_t max_n;
-};
-constexpr int kSortItems = 64;                 // items per lane per tile
-constexpr int kSortTile = 32 * kSortItems;     // elements per warp tile
+// Stable LSD radix sort of (u64 key, u32 value) pairs, 8-bit digits, `bits` low key bits.
+// Keys travel with values, so every pass reads and writes contiguously.
+constexpr int kSortThreads = 256;
+constexpr int kSortItems = 16;                              // per lane
+constexpr int kSortTile = kSortThreads * kSortItems;        // 4096 elements per block tile
 inline uint64_t sort_tiles(uint64_t n) { return (n + kSortTile - 1) / kSortTile; }
-struct Q18SortSpec {         // host-computed from Q18Stats
-    long long amt_max, ent_min; int w_min, d_min, o_min; long long nd, no;  // dense rowkey
-    int bits[3];             // field 0: rowkey (asc), 1: entry (asc), 2: amount (desc)
+struct SortPairs {
+    unsigned long long *k[2];
+    unsigned int *v[2];
+    unsigned int *counts;        // [256 * tiles]
+    unsigned int *totals;        // [256]
 };
-void launch_q18_sort_keys(const Q18Cols &cols, uint64_t n, const Q18SortSpec &spec,
-                          const SortScratch &s, int num_sms, cudaStream_t st);
-// Sorts; returns the buffer holding the final permutation.
-unsigned int *radix_sort_fields(uint64_t n, const int bits[3], const SortScratch &s,
-                                cudaStream_t st, int num_sms);
-void launch_q18_permute(const Q18Cols &src, const unsigned int *perm, uint64_t n,
+// Returns which buffer (0/1) holds the sorted pairs (input is in k[0]/v[0]).
+int radix_sort_pairs(uint64_t n, int bits, const SortPairs &s, int num_sms, cudaStream_t st);
+
+// Q18 ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id (R11).
+struct Q18SortSpec {         // host-computed from Q18Stats
+    long long amt_max, ent_min;
+    int w_min, d_min, o_min;
+    long long nd, no;        // extents of d and o (dense row rank)
+    int bits_a, bits_e, bits_r;  // field widths: amount (desc), entry, row rank
+    int prefix_bits;         // width of the sorted 64-bit prefix of the composite key
+};
+void launch_q18_sort_keys(const Q18Row *rows, uint64_t n, const Q18SortSpec &spec,
+                          const SortPairs &s, int num_sms, cudaStream_t st);
+// Within runs of equal prefix, order by the full tuple; runs longer than 32 raise *flag.
+void launch_q18_tiefix(const Q18Row *rows, const unsigned long long *keys, unsigned int *vals,
+                       uint64_t n, unsigned int *flag, int num_sms, cudaStream_t st);
+// Exact fallback: three stable passes over the full fields (row rank, entry, amount).
+void launch_q18_field_keys(const Q18Row *rows, const unsigned int *vals, uint64_t n, int field,
+                           const Q18SortSpec &spec, unsigned long long *keys, int num_sms,
+                           cudaStream_t st);
+void launch_iota(unsigned int *v, uint64_t n, int num_sms, cudaStream_t st);
+void launch_q18_permute(const Q18Row *rows, const unsigned int *perm, uint64_t n,
                         const Q18Cols &dst, int num_sms, cudaStream_t st);
+
+// ------------------------------------------------------------ store (a1) --
+void launch_stats_init(int *out, int n_pairs, cudaStream_t st);  // pairs of (INT_MAX, INT_MIN)
+void launch_minmax_i32(const int32_t *p, uint64_t n, int *out, int num_sms, cudaStream_t st);
 
 // ---------------------------------------------------------------- helpers --
 // Every launcher counts the kernels it launches (reported per query as kernel_launches).
 void count_launches(int n);
 uint64_t launches_total();
-void launch_fill_u64(unsigned long long *p, uint64_t n, unsigned long long v, cudaStream_t st);
 
 }  // namespace h2tap

@@ -1,14 +1,15 @@
 // sort_kernels.cu — a8 finalize for CH Q18: ORDER BY amount_sum DESC, o_entry_d ASC, then the
-// (o_w_id, o_d_id, o_id) tie-break (R11), as a stable LSD radix sort of a permutation.
+// (o_w_id, o_d_id, o_id) tie-break that makes the order total (R11).
 //
-// Each sort field is mapped to an unsigned key whose bit width is taken from the data's
-// min/max (computed by the HAVING kernel), so only the passes the data needs are run:
-//   field 0 (least significant): dense rank of (w, d, o)  asc
-//   field 1:                      o_entry_d - min          asc
-//   field 2 (most significant):  max - amount_sum          (= DESC)
-// One pass = histogram (per 8192-element block tile) -> exclusive scan -> stable scatter.
-// Stability inside a tile comes from processing each warp's sub-tile in order with
-// __match_any_sync ranks, and tiles in order via the digit-major count layout.
+// The three sort fields are mapped to unsigned integers whose widths come from the result's
+// min/max (HAVING kernel statistics): a = max - amount_sum (DESC), e = o_entry_d - min,
+// r = dense rank of (w, d, o). Their concatenation a|e|r is the exact composite key.
+//  * composite <= 64 bits: one stable LSD radix sort of (key, row) pairs — exact.
+//  * wider: sort by the composite's top `prefix_bits`, then order each run of equal prefixes by
+//    the full tuple (runs are a handful of rows on realistic data); a run longer than 32 rows
+//    raises a flag and the engine redoes the sort exactly, field by field (r, then e, then a).
+// Radix pass = per-tile digit histogram -> per-digit scan -> stable scatter; keys travel with
+// their row ids so every pass reads and writes contiguous arrays.
 #include <cstdint>
 #include <cuda_runtime.h>
 
@@ -18,51 +19,47 @@ namespace h2tap {
 namespace {
 
 constexpr unsigned kFull = 0xffffffffu;
-constexpr int kThreads = 256;
-constexpr int kWarps = kThreads / 32;
-constexpr int kItems = 32;                       // per lane per block tile
-constexpr int kWarpTile = 32 * kItems;           // 1024
-constexpr int kBlockTile = kWarps * kWarpTile;   // 8192
+constexpr int kT = kSortThreads;         // 256
+constexpr int kI = kSortItems;           // 16
+constexpr int kWarps = kT / 32;
+constexpr int kWarpTile = 32 * kI;       // 512
 
-__device__ __forceinline__ unsigned int digit_of(const unsigned long long *__restrict__ key,
-                                                 const unsigned int *__restrict__ idx,
-                                                 uint64_t j, int shift) {
-    const unsigned int e = idx ? idx[j] : (unsigned int)j;
-    return (unsigned int)(__ldcg(key + e) >> shift) & 0xffu;
-}
-
-__global__ void __launch_bounds__(kThreads)
-hist_kernel(const unsigned long long *__restrict__ key, const unsigned int *__restrict__ idx,
-            uint64_t n, int shift, unsigned int *__restrict__ counts, uint64_t ntiles) {
+// ------------------------------------------------------------- radix pass --
+__global__ void __launch_bounds__(kT)
+hist_kernel(const unsigned long long *__restrict__ key, uint64_t n, int shift,
+            unsigned int *__restrict__ counts, uint64_t ntiles) {
     __shared__ unsigned int h[256];
-    for (int i = threadIdx.x; i < 256; i += kThreads) h[i] = 0;
+    for (int i = threadIdx.x; i < 256; i += kT) h[i] = 0;
     __syncthreads();
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    const uint64_t base = (uint64_t)blockIdx.x * kBlockTile + (uint64_t)warp * kWarpTile;
-    for (int it = 0; it < kItems; ++it) {
-        const uint64_t j = base + it * 32 + lane;
-        const bool ok = j < n;
-        const unsigned int dg = ok ? digit_of(key, idx, j, shift) : 256u + lane;  // unique dummy
-        const unsigned int peers = __match_any_sync(kFull, dg);
-        if (ok && lane == __ffs(peers) - 1) atomicAdd(&h[dg], (unsigned int)__popc(peers));
+    const uint64_t base = (uint64_t)blockIdx.x * kSortTile + (uint64_t)warp * kWarpTile + lane;
+    unsigned int dg[kI];
+#pragma unroll
+    for (int i = 0; i < kI; ++i) {
+        const uint64_t j = base + i * 32;
+        dg[i] = j < n ? (unsigned int)(__ldcg(key + j) >> shift) & 0xffu : 256u + lane;  // unique dummy
+    }
+#pragma unroll
+    for (int i = 0; i < kI; ++i) {
+        const unsigned int peers = __match_any_sync(kFull, dg[i]);
+        if (dg[i] < 256u && lane == __ffs(peers) - 1) atomicAdd(&h[dg[i]], (unsigned int)__popc(peers));
     }
     __syncthreads();
-    for (int d = threadIdx.x; d < 256; d += kThreads) counts[(uint64_t)d * ntiles + blockIdx.x] = h[d];
+    for (int d = threadIdx.x; d < 256; d += kT) counts[(uint64_t)d * ntiles + blockIdx.x] = h[d];
 }
 
-// Exclusive scan of `len` counts in place, one block of 1024 threads, coalesced rounds.
-__global__ void __launch_bounds__(1024) scan_kernel(unsigned int *__restrict__ c, uint64_t len) {
-    __shared__ unsigned int wsum[32];
-    __shared__ unsigned int carry_s;
+// One block per digit: exclusive scan of that digit's per-tile counts, total -> totals[d].
+__global__ void __launch_bounds__(256) digit_scan_kernel(unsigned int *__restrict__ counts,
+                                                         uint64_t ntiles,
+                                                         unsigned int *__restrict__ totals) {
+    __shared__ unsigned int wsum[8];
+    unsigned int *row = counts + (uint64_t)blockIdx.x * ntiles;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     unsigned int carry = 0;
-    for (uint64_t r0 = 0; r0 < len; r0 += 4096) {
-        unsigned int v[4];
-        const uint64_t b = r0 + 4 * (uint64_t)threadIdx.x;
-#pragma unroll
-        for (int k = 0; k < 4; ++k) v[k] = b + k < len ? c[b + k] : 0u;
-        const unsigned int s = v[0] + v[1] + v[2] + v[3];
-        unsigned int x = s;  // inclusive warp scan
+    for (uint64_t r0 = 0; r0 < ntiles; r0 += 256) {
+        const uint64_t i = r0 + threadIdx.x;
+        const unsigned int v = i < ntiles ? row[i] : 0u;
+        unsigned int x = v;
 #pragma unroll
         for (int o = 1; o < 32; o <<= 1) {
             const unsigned int t = __shfl_up_sync(kFull, x, o);
@@ -70,96 +67,196 @@ __global__ void __launch_bounds__(1024) scan_kernel(unsigned int *__restrict__ c
         }
         if (lane == 31) wsum[warp] = x;
         __syncthreads();
-        if (warp == 0) {
-            unsigned int y = wsum[lane];
+        unsigned int before = 0, all = 0;
 #pragma unroll
-            for (int o = 1; o < 32; o <<= 1) {
-                const unsigned int t = __shfl_up_sync(kFull, y, o);
-                if (lane >= o) y += t;
-            }
-            wsum[lane] = y;  // inclusive over warps
-            if (lane == 31) carry_s = y;
+        for (int w = 0; w < 8; ++w) {
+            before += w < warp ? wsum[w] : 0u;
+            all += wsum[w];
         }
-        __syncthreads();
-        unsigned int ex = carry + (warp ? wsum[warp - 1] : 0u) + x - s;
-#pragma unroll
-        for (int k = 0; k < 4; ++k) {
-            if (b + k < len) c[b + k] = ex;
-            ex += v[k];
-        }
-        carry += carry_s;
+        if (i < ntiles) row[i] = carry + before + x - v;
+        carry += all;
         __syncthreads();
     }
+    if (threadIdx.x == 0) totals[blockIdx.x] = carry;
 }
 
-__global__ void __launch_bounds__(kThreads)
-scatter_kernel(const unsigned long long *__restrict__ key, const unsigned int *__restrict__ idx_in,
-               unsigned int *__restrict__ idx_out, uint64_t n, int shift,
-               const unsigned int *__restrict__ offsets, uint64_t ntiles) {
-    __shared__ unsigned int wcount[kWarps][256];  // per-warp digit counts -> running offsets
+__global__ void __launch_bounds__(kT)
+scatter_kernel(const unsigned long long *__restrict__ kin, const unsigned int *__restrict__ vin,
+               unsigned long long *__restrict__ kout, unsigned int *__restrict__ vout, uint64_t n,
+               int shift, const unsigned int *__restrict__ counts, uint64_t ntiles,
+               const unsigned int *__restrict__ totals) {
+    __shared__ unsigned int wc[kWarps][256];  // per-warp digit counts -> running offsets
+    __shared__ unsigned int dbase[256];
+    __shared__ unsigned int ws[kWarps];
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    for (int i = threadIdx.x; i < kWarps * 256; i += kThreads) (&wcount[0][0])[i] = 0;
-    __syncthreads();
-    const uint64_t base = (uint64_t)blockIdx.x * kBlockTile + (uint64_t)warp * kWarpTile;
-    for (int it = 0; it < kItems; ++it) {  // pass 1: per-warp histogram
-        const uint64_t j = base + it * 32 + lane;
-        const bool ok = j < n;
-        const unsigned int dg = ok ? digit_of(key, idx_in, j, shift) : 256u + lane;
-        const unsigned int peers = __match_any_sync(kFull, dg);
-        if (ok && lane == __ffs(peers) - 1) wcount[warp][dg] += __popc(peers);
+    for (int i = threadIdx.x; i < kWarps * 256; i += kT) (&wc[0][0])[i] = 0;
+    {   // exclusive scan of the 256 digit totals (every block recomputes it: 256 values)
+        const unsigned int v = totals[threadIdx.x];
+        unsigned int x = v;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const unsigned int t = __shfl_up_sync(kFull, x, o);
+            if (lane >= o) x += t;
+        }
+        if (lane == 31) ws[warp] = x;
+        __syncthreads();
+        unsigned int before = 0;
+        for (int w = 0; w < warp; ++w) before += ws[w];
+        dbase[threadIdx.x] = before + x - v;
+    }
+    const uint64_t base = (uint64_t)blockIdx.x * kSortTile + (uint64_t)warp * kWarpTile + lane;
+    unsigned long long k[kI];
+    unsigned int v[kI], dg[kI];
+#pragma unroll
+    for (int i = 0; i < kI; ++i) {
+        const uint64_t j = base + i * 32;
+        if (j < n) {
+            k[i] = __ldcs(kin + j);
+            v[i] = __ldcs(vin + j);
+            dg[i] = (unsigned int)(k[i] >> shift) & 0xffu;
+        } else {
+            k[i] = 0; v[i] = 0; dg[i] = 256u + lane;
+        }
     }
     __syncthreads();
-    // running offset of warp w for digit d = tile offset[d] + counts of warps < w
-    for (int d = threadIdx.x; d < 256; d += kThreads) {
-        unsigned int run = offsets[(uint64_t)d * ntiles + blockIdx.x];
+    unsigned int peers[kI];
+#pragma unroll
+    for (int i = 0; i < kI; ++i) {  // per-warp histogram (leaders only; __syncwarp orders RAW)
+        peers[i] = __match_any_sync(kFull, dg[i]);
+        if (dg[i] < 256u && lane == __ffs(peers[i]) - 1) wc[warp][dg[i]] += __popc(peers[i]);
+        __syncwarp();
+    }
+    __syncthreads();
+    {   // running offset of warp w for digit d = global digit base + tile offset + warps < w
+        const int d = threadIdx.x;
+        unsigned int run = dbase[d] + counts[(uint64_t)d * ntiles + blockIdx.x];
+#pragma unroll
         for (int w = 0; w < kWarps; ++w) {
-            const unsigned int c = wcount[w][d];
-            wcount[w][d] = run;
+            const unsigned int c = wc[w][d];
+            wc[w][d] = run;
             run += c;
         }
     }
     __syncthreads();
     const unsigned lt = (1u << lane) - 1u;
-    for (int it = 0; it < kItems; ++it) {  // pass 2: stable scatter in (iteration, lane) order
-        const uint64_t j = base + it * 32 + lane;
-        const bool ok = j < n;
-        const unsigned int dg = ok ? digit_of(key, idx_in, j, shift) : 256u + lane;
-        const unsigned int peers = __match_any_sync(kFull, dg);
-        if (ok) {
-            const unsigned int pos = wcount[warp][dg] + __popc(peers & lt);
-            idx_out[pos] = idx_in ? idx_in[j] : (unsigned int)j;
+#pragma unroll
+    for (int i = 0; i < kI; ++i) {  // stable scatter in (warp, item, lane) = index order
+        if (dg[i] < 256u) {
+            const unsigned int pos = wc[warp][dg[i]] + __popc(peers[i] & lt);
+            kout[pos] = k[i];
+            vout[pos] = v[i];
         }
         __syncwarp();
-        if (ok && lane == __ffs(peers) - 1) wcount[warp][dg] += __popc(peers);
+        if (dg[i] < 256u && lane == __ffs(peers[i]) - 1) wc[warp][dg[i]] += __popc(peers[i]);
         __syncwarp();
     }
 }
 
-__global__ void sort_keys_kernel(Q18Cols c, uint64_t n, Q18SortSpec sp, SortScratch s) {
+// ------------------------------------------------------------ Q18 keys --
+__device__ __forceinline__ unsigned long long field_a(const Q18Row &r, const Q18SortSpec &sp) {
+    return (unsigned long long)sp.amt_max - (unsigned long long)r.amount_sum;  // DESC
+}
+__device__ __forceinline__ unsigned long long field_e(const Q18Row &r, const Q18SortSpec &sp) {
+    return (unsigned long long)r.o_entry_d - (unsigned long long)sp.ent_min;
+}
+__device__ __forceinline__ unsigned long long field_r(const Q18Row &r, const Q18SortSpec &sp) {
+    const unsigned long long w = (unsigned)(r.o_w_id - sp.w_min);
+    const unsigned long long d = (unsigned)(r.o_d_id - sp.d_min);
+    const unsigned long long o = (unsigned)(r.o_id - sp.o_min);
+    return (w * (unsigned long long)sp.nd + d) * (unsigned long long)sp.no + o;
+}
+
+// top `prefix_bits` bits of the concatenation (a | e | r) with widths (bits_a, bits_e, bits_r)
+__device__ __forceinline__ unsigned long long prefix_key(const Q18Row &r, const Q18SortSpec &sp) {
+    const unsigned long long f[3] = {field_a(r, sp), field_e(r, sp), field_r(r, sp)};
+    const int b[3] = {sp.bits_a, sp.bits_e, sp.bits_r};
+    unsigned long long p = 0;
+    int room = sp.prefix_bits;
+#pragma unroll
+    for (int i = 0; i < 3; ++i) {
+        const int take = b[i] < room ? b[i] : room;
+        if (take > 0) {
+            p = (take == 64 ? 0ull : (p << take)) | (f[i] >> (b[i] - take));
+            room -= take;
+        }
+    }
+    return p;
+}
+
+__global__ void sort_keys_kernel(const Q18Row *__restrict__ rows, uint64_t n, Q18SortSpec sp,
+                                 unsigned long long *__restrict__ k, unsigned int *__restrict__ v) {
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
-        const unsigned long long w = (unsigned)(c.o_w_id[i] - sp.w_min);
-        const unsigned long long d = (unsigned)(c.o_d_id[i] - sp.d_min);
-        const unsigned long long o = (unsigned)(c.o_id[i] - sp.o_min);
-        s.key[0][i] = (w * (unsigned long long)sp.nd + d) * (unsigned long long)sp.no + o;
-        s.key[1][i] = (unsigned long long)c.o_entry_d[i] - (unsigned long long)sp.ent_min;
-        s.key[2][i] = (unsigned long long)sp.amt_max - (unsigned long long)c.amount_sum[i];
+        k[i] = prefix_key(rows[i], sp);
+        v[i] = (unsigned int)i;
     }
 }
 
-__global__ void permute_kernel(Q18Cols src, const unsigned int *__restrict__ perm, uint64_t n,
-                               Q18Cols dst) {
+// full ORDER BY comparison: amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id
+__device__ __forceinline__ bool row_less(const Q18Row &x, const Q18Row &y) {
+    if (x.amount_sum != y.amount_sum) return x.amount_sum > y.amount_sum;
+    if (x.o_entry_d != y.o_entry_d) return x.o_entry_d < y.o_entry_d;
+    if (x.o_w_id != y.o_w_id) return x.o_w_id < y.o_w_id;
+    if (x.o_d_id != y.o_d_id) return x.o_d_id < y.o_d_id;
+    return x.o_id < y.o_id;
+}
+
+constexpr int kMaxRun = 32;
+
+__global__ void tiefix_kernel(const Q18Row *__restrict__ rows, const unsigned long long *__restrict__ k,
+                              unsigned int *__restrict__ v, uint64_t n, unsigned int *flag) {
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
+        const unsigned long long ki = k[i];
+        if (i > 0 && k[i - 1] == ki) continue;         // not the head of a run
+        if (i + 1 >= n || k[i + 1] != ki) continue;    // run of one
+        uint64_t j = i + 1;
+        while (j < n && k[j] == ki && j - i <= kMaxRun) ++j;
+        if (j - i > kMaxRun) { atomicOr(flag, 1u); continue; }
+        unsigned int idx[kMaxRun];
+        const int len = (int)(j - i);
+        for (int t = 0; t < len; ++t) idx[t] = v[i + t];
+        for (int t = 1; t < len; ++t) {  // insertion sort by the full tuple
+            const unsigned int x = idx[t];
+            const Q18Row rx = rows[x];
+            int u = t - 1;
+            while (u >= 0 && row_less(rx, rows[idx[u]])) { idx[u + 1] = idx[u]; --u; }
+            idx[u + 1] = x;
+        }
+        for (int t = 0; t < len; ++t) v[i + t] = idx[t];
+    }
+}
+
+__global__ void field_keys_kernel(const Q18Row *__restrict__ rows, const unsigned int *__restrict__ vals,
+                                  uint64_t n, int field, Q18SortSpec sp,
+                                  unsigned long long *__restrict__ k) {
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
+        const Q18Row r = rows[vals[i]];
+        k[i] = field == 0 ? field_r(r, sp) : field == 1 ? field_e(r, sp) : field_a(r, sp);
+    }
+}
+
+__global__ void iota_kernel(unsigned int *v, uint64_t n) {
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride)
+        v[i] = (unsigned int)i;
+}
+
+// Gather one 40-byte row per output position, write the eight SoA columns coalesced.
+__global__ void permute_kernel(const Q18Row *__restrict__ rows, const unsigned int *__restrict__ perm,
+                               uint64_t n, Q18Cols dst) {
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < n; j += stride) {
-        const unsigned int i = perm ? perm[j] : (unsigned int)j;
-        dst.c_last[j] = src.c_last[i];
-        dst.c_id[j] = src.c_id[i];
-        dst.o_id[j] = src.o_id[i];
-        dst.o_entry_d[j] = src.o_entry_d[i];
-        dst.o_ol_cnt[j] = src.o_ol_cnt[i];
-        dst.amount_sum[j] = src.amount_sum[i];
-        dst.o_w_id[j] = src.o_w_id[i];
-        dst.o_d_id[j] = src.o_d_id[i];
+        const Q18Row r = rows[perm ? perm[j] : j];
+        dst.c_last[j] = r.c_last;
+        dst.c_id[j] = r.c_id;
+        dst.o_id[j] = r.o_id;
+        dst.o_entry_d[j] = r.o_entry_d;
+        dst.o_ol_cnt[j] = r.o_ol_cnt;
+        dst.amount_sum[j] = r.amount_sum;
+        dst.o_w_id[j] = r.o_w_id;
+        dst.o_d_id[j] = r.o_d_id;
     }
 }
 
@@ -172,38 +269,50 @@ unsigned grid_cap(uint64_t work, int threads, int num_sms, int per_sm) {
 
 }  // namespace
 
-void launch_q18_sort_keys(const Q18Cols &cols, uint64_t n, const Q18SortSpec &spec,
-                          const SortScratch &s, int num_sms, cudaStream_t st) {
-    sort_keys_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(cols, n, spec, s);
+int radix_sort_pairs(uint64_t n, int bits, const SortPairs &s, int num_sms, cudaStream_t st) {
+    (void)num_sms;
+    const uint64_t ntiles = sort_tiles(n);
+    int cur = 0;
+    for (int shift = 0; shift < bits; shift += 8) {
+        hist_kernel<<<(unsigned)ntiles, kT, 0, st>>>(s.k[cur], n, shift, s.counts, ntiles);
+        count_launches(1);
+        digit_scan_kernel<<<256, 256, 0, st>>>(s.counts, ntiles, s.totals);
+        count_launches(1);
+        scatter_kernel<<<(unsigned)ntiles, kT, 0, st>>>(s.k[cur], s.v[cur], s.k[cur ^ 1], s.v[cur ^ 1],
+                                                         n, shift, s.counts, ntiles, s.totals);
+        count_launches(1);
+        cur ^= 1;
+    }
+    return cur;
+}
+
+void launch_q18_sort_keys(const Q18Row *rows, uint64_t n, const Q18SortSpec &spec,
+                          const SortPairs &s, int num_sms, cudaStream_t st) {
+    sort_keys_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, n, spec, s.k[0], s.v[0]);
     count_launches(1);
 }
 
-unsigned int *radix_sort_fields(uint64_t n, const int bits[3], const SortScratch &s,
-                                cudaStream_t st, int num_sms) {
-    (void)num_sms;
-    const uint64_t ntiles = (n + kBlockTile - 1) / kBlockTile;
-    const unsigned int *in = nullptr;  // identity permutation before the first pass
-    unsigned int *out = s.idx_a;
-    for (int f = 0; f < 3; ++f) {
-        for (int shift = 0; shift < bits[f]; shift += 8) {
-            hist_kernel<<<(unsigned)ntiles, kThreads, 0, st>>>(s.key[f], in, n, shift, s.counts, ntiles);
-            count_launches(1);
-            scan_kernel<<<1, 1024, 0, st>>>(s.counts, 256 * ntiles);
-            count_launches(1);
-            scatter_kernel<<<(unsigned)ntiles, kThreads, 0, st>>>(s.key[f], in, out, n, shift, s.counts,
-                                                                ntiles);
-            count_launches(1);
-            in = out;
-            out = (out == s.idx_a) ? s.idx_b : s.idx_a;
-        }
-    }
-    // nullptr = zero passes were needed (n <= 1 or all keys equal): identity permutation
-    return const_cast<unsigned int *>(in);
+void launch_q18_tiefix(const Q18Row *rows, const unsigned long long *keys, unsigned int *vals,
+                       uint64_t n, unsigned int *flag, int num_sms, cudaStream_t st) {
+    tiefix_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, keys, vals, n, flag);
+    count_launches(1);
 }
 
-void launch_q18_permute(const Q18Cols &src, const unsigned int *perm, uint64_t n,
+void launch_q18_field_keys(const Q18Row *rows, const unsigned int *vals, uint64_t n, int field,
+                           const Q18SortSpec &spec, unsigned long long *keys, int num_sms,
+                           cudaStream_t st) {
+    field_keys_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, vals, n, field, spec, keys);
+    count_launches(1);
+}
+
+void launch_iota(unsigned int *v, uint64_t n, int num_sms, cudaStream_t st) {
+    iota_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(v, n);
+    count_launches(1);
+}
+
+void launch_q18_permute(const Q18Row *rows, const unsigned int *perm, uint64_t n,
                         const Q18Cols &dst, int num_sms, cudaStream_t st) {
-    permute_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(src, perm, n, dst);
+    permute_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, perm, n, dst);
     count_launches(1);
 }
 

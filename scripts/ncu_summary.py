@@ -1,0 +1,56 @@
+"""Summarise an ncu launch list (--metrics gpu__time_duration.sum csv) and a --set full report
+into a markdown table under profiles/. Usage: python scripts/ncu_summary.py <tag>"""
+import collections
+import csv
+import json
+import os
+import subprocess
+import sys
+
+tag = sys.argv[1]
+root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+out = []
+lp = os.path.join(root, "gpurun_out", f"launches_{tag}.csv")
+if os.path.exists(lp):
+    rows = list(csv.reader(open(lp)))
+    hdr = next(i for i, r in enumerate(rows) if "Kernel Name" in r)
+    H = rows[hdr]
+    ki, vi = H.index("Kernel Name"), H.index("Metric Value")
+    agg = collections.OrderedDict()
+    for r in rows[hdr + 1:]:
+        if len(r) > vi:
+            agg.setdefault(r[ki].split("(")[0].split("::")[-1], []).append(float(r[vi].replace(",", "")))
+    tot = sum(sum(v) for v in agg.values())
+    out.append(f"## Launch list ({lp.split('/')[-1]}, ncu gpu__time_duration.sum, cold cache, serialised)\n")
+    out.append("| kernel | launches | mean us | share of listed time |\n|---|---|---|---|")
+    for k, v in agg.items():
+        out.append(f"| {k} | {len(v)} | {sum(v)/len(v)/1e3:.1f} | {sum(v)/tot:.3f} |")
+rp = os.path.join(root, "gpurun_out", f"prof_{tag}.ncu-rep")
+traffic = {}
+if os.path.exists(rp):
+    raw = subprocess.run(["ncu", "-i", rp, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
+    r = list(csv.reader(raw.splitlines()))
+    h = r[0]
+    want = ["Kernel Name", "gpu__time_duration.sum", "dram__bytes_read.sum", "dram__bytes_write.sum",
+            "gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed",
+            "sm__throughput.avg.pct_of_peak_sustained_elapsed", "launch__registers_per_thread",
+            "sm__warps_active.avg.pct_of_peak_sustained_active", "lts__t_sector_hit_rate.pct"]
+    idx = [h.index(w) for w in want if w in h]
+    out.append(f"\n## ncu --set full ({rp.split('/')[-1]})\n")
+    out.append("| " + " | ".join(h[i] for i in idx) + " |")
+    out.append("|" + "---|" * len(idx))
+    out.append("| " + " | ".join(r[1][i] for i in idx) + " |")
+    unit = {h[i]: r[1][i] for i in idx}
+    for row in r[2:]:
+        name = row[h.index("Kernel Name")].split("(")[0].split("::")[-1]
+        out.append("| " + " | ".join([name] + [row[i] for i in idx[1:]]) + " |")
+        mult = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9}
+        rd = float(row[h.index("dram__bytes_read.sum")]) * mult[unit["dram__bytes_read.sum"]]
+        wr = float(row[h.index("dram__bytes_write.sum")]) * mult[unit["dram__bytes_write.sum"]]
+        traffic.setdefault(name, []).append(rd + wr)
+md = os.path.join(root, "profiles", f"{tag}_ncu_summary.md")
+open(md, "w").write(f"# ncu summary {tag}\n\n" + "\n".join(out) + "\n")
+print(open(md).read())
+if traffic:
+    tj = os.path.join(root, "profiles", f"{tag}_traffic.json")
+    json.dump({k: sum(v) / len(v) for k, v in traffic.items()}, open(tj, "w"), indent=1)

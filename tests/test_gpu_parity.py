@@ -16,6 +16,7 @@ import oracle
 from chref import (Q1_CUTOFF, Q6_D_HI, Q6_D_LO, Q6_Q_HI, Q6_Q_LO, Q18_HAVING, golden, iso_us)
 
 pytestmark = pytest.mark.gpu
+HASH = 4  # H2TAP_QUERY_HASH_JOIN
 
 Q18_NAMES = ["c_last", "c_id", "o_id", "o_entry_d", "o_ol_cnt", "amount_sum", "o_w_id", "o_d_id"]
 Q1_NAMES = ["ol_number", "sum_qty", "sum_amount", "avg_qty", "avg_amount", "count_order"]
@@ -89,8 +90,10 @@ def run_all(L, t, rng=None, n_rand=2):
     assert_q6(L.q(6), oracle.q6(t, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))  # CH defaults in the library
     assert_q1(L.q(1, [Q1_CUTOFF]), oracle.q1(t, Q1_CUTOFF))
     assert_q1(L.q(1), oracle.q1(t, Q1_CUTOFF))
-    assert_q18(L.q(18, [Q18_HAVING]), oracle.q18(t, Q18_HAVING))
-    assert_q18(L.q(18), oracle.q18(t, Q18_HAVING))
+    want18 = oracle.q18(t, Q18_HAVING)
+    assert_q18(L.q(18, [Q18_HAVING]), want18)
+    assert_q18(L.q(18), want18)
+    assert_q18(L.q(18, flags=HASH), want18)  # open-addressing join indexes forced
     rng = rng or np.random.default_rng(0)
     for _ in range(n_rand):
         d_lo = int(rng.integers(chgen.TS_1995, chgen.TS_2025))
@@ -100,7 +103,9 @@ def run_all(L, t, rng=None, n_rand=2):
         cut = int(rng.integers(chgen.TS_1995, chgen.TS_2025))
         assert_q1(L.q(1, [cut]), oracle.q1(t, cut))
         thr = int(rng.integers(-10, 8_000_000))
-        assert_q18(L.q(18, [thr]), oracle.q18(t, thr))
+        want18 = oracle.q18(t, thr)
+        assert_q18(L.q(18, [thr]), want18)
+        assert_q18(L.q(18, [thr], flags=HASH), want18)
 
 
 # ----------------------------------------------------------------- cases --
@@ -185,7 +190,9 @@ def test_q18_join_edges(L):
     t["orders"] = {k: v[mask].copy() for k, v in o.items()}
     L.load(t)
     for thr in (-1, 0, Q18_HAVING, 4_000_000):
-        assert_q18(L.q(18, [thr]), oracle.q18(t, thr))
+        want = oracle.q18(t, thr)
+        assert_q18(L.q(18, [thr]), want)
+        assert_q18(L.q(18, [thr], flags=HASH), want)
 
 
 def test_q18_ties_use_full_order(L):
@@ -198,6 +205,43 @@ def test_q18_ties_use_full_order(L):
         assert_q18(L.q(18, [thr]), oracle.q18(t, thr))
 
 
+def test_q18_sort_fallback_long_prefix_runs(L):
+    """Composite key > 64 bits and > 32 rows sharing the 48-bit prefix: exact field-by-field
+    re-sort path."""
+    t = chgen.generate(1, 3, seed=17)
+    t["order_line"]["ol_amount"][:] = 1000            # amount_sum in {5000, ..., 15000}
+    o = t["orders"]
+    half = np.arange(len(o["o_id"])) % 2 == 0
+    o["o_entry_d"][half] = chgen.TS_2025 - 10**6 + (np.arange(int(half.sum())) % 1000)
+    L.load(t)
+    for thr in (0, 9000):
+        want = oracle.q18(t, thr)
+        assert_q18(L.q(18, [thr]), want)
+        assert_q18(L.q(18, [thr], flags=HASH), want)
+
+
+def test_q18_planner_dense_and_hash(h, eng, L):
+    """TPC-C keys are dense -> perfect-hash indexes; sparse keys -> open addressing."""
+    t = chgen.generate(1, 3, seed=19)
+    L.load(t)
+    r = h.h2tap_run_query(eng, h.H2TAP_Q18)
+    assert r.plan_flags == 3
+    r.free()
+    r = h.h2tap_run_query(eng, h.H2TAP_Q18, flags=HASH)
+    assert r.plan_flags == 0
+    r.free()
+    for tab, col in (("orders", "o_id"), ("order_line", "ol_o_id")):
+        t[tab][col] = t[tab][col] * 1000 + 7         # same join, sparse key box
+    t["customer"]["c_id"] = t["customer"]["c_id"] * 977
+    t["orders"]["o_c_id"] = t["orders"]["o_c_id"] * 977
+    L.load(t)
+    r = h.h2tap_run_query(eng, h.H2TAP_Q18)
+    got = r.to_numpy()
+    assert r.plan_flags == 0
+    r.free()
+    assert_q18(got, oracle.q18(t, Q18_HAVING))
+
+
 def test_q18_duplicate_key_rejected(h, L):
     t = chgen.generate(1, 2, seed=2)
     o = t["orders"]
@@ -206,6 +250,9 @@ def test_q18_duplicate_key_rejected(h, L):
     L.load(t)
     with pytest.raises(h.H2tapError) as ei:
         L.q(18)
+    assert ei.value.status == h.H2TAP_EDUPKEY
+    with pytest.raises(h.H2tapError) as ei:
+        L.q(18, flags=HASH)
     assert ei.value.status == h.H2TAP_EDUPKEY
     assert_q6(L.q(6), oracle.q6(t, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))  # engine still usable
 
@@ -372,7 +419,8 @@ def test_full_size_w100_bench_config(h, w100):
         L = Loader(h, e)
         assert_q6(L.q(6), oracle.q6(w100, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))
         assert_q1(L.q(1), oracle.q1(w100, Q1_CUTOFF))
-        got = L.q(18, flags=h.H2TAP_QUERY_PROFILE)
-        assert_q18(got, oracle.q18(w100, Q18_HAVING))
+        want = oracle.q18(w100, Q18_HAVING)
+        assert_q18(L.q(18, flags=h.H2TAP_QUERY_PROFILE), want)
+        assert_q18(L.q(18, flags=HASH), want)
     finally:
         h.h2tap_close(e)
