@@ -135,7 +135,8 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes):
         "q18_probe_groupjoin": 20 * n_ol + 16 * n_o + 16 * n_o,
         "q18_having_compact": 16 * n_o + 28 * n_o + 16 * n_pass + 4 * n_pass + 40 * n_pass,
         "q18_sort_keys": 40 * n_pass + 24 * n_pass,
-        "q18_radix_sort": sort_passes * (2 * (4 + 8) + 4 + 4) * n_pass,
+        "q18_bucket_sort": (8 + 12 + 12 + 12 + 12) * n_pass,
+        "q18_tiefix": 8 * n_pass,
         "q18_permute": (4 + 40 + 40) * n_pass,
     }.get(kernel)
 
@@ -281,9 +282,7 @@ def main():
 
     # ---- roofline for the dominant kernel (largest share of the step)
     kavg = {k: float(np.mean(v)) for k, v in kern.items()}
-    # radix passes (3 kernels each) are folded into q18_radix_sort; recover the pass count from
-    # the query's launch count: init, build, probe, having, sort_keys, permute + 3 per pass
-    sort_passes = max(0, (q18_launches - 6) // 3)
+    sort_passes = 0
     dominant = max(kavg, key=kavg.get) if kavg else None
     peak, peak_src = peaks()
     roof = None
@@ -300,7 +299,7 @@ def main():
     for k, v in kavg.items():
         b = alg_bytes(k, n_ol, n_o, n_c, n_pass, sort_passes)
         kernels_summary[k] = {"ms": round(v, 5), "share": round(v / step_ms_local, 4)}
-        if b and k != "q18_radix_sort":
+        if b:
             kernels_summary[k]["GB/s"] = round(b / (v / 1e3) / 1e9, 1)
             kernels_summary[k]["frac_hbm"] = round(b / (v / 1e3) / 1e9 / peak, 4)
 

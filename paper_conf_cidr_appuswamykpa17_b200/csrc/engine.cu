@@ -841,7 +841,7 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
         sp.bits_e = bitwidth((unsigned long long)st.ent_max - (unsigned long long)st.ent_min);
         sp.bits_r = bitwidth(nw * (unsigned long long)sp.nd * (unsigned long long)sp.no - 1);
         const int B = sp.bits_a + sp.bits_e + sp.bits_r;
-        sp.prefix_bits = B <= 64 ? B : 48;
+        sp.prefix_bits = B <= 64 ? B : 64;
         tiefix = B > sp.prefix_bits;
         for (int b = 0; b < 2; ++b) {
             sp2.k[b] = static_cast<unsigned long long *>(e->arena.get("q18.sk" + std::to_string(b), 8 * nout));
@@ -849,16 +849,24 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
         }
         sp2.counts = static_cast<unsigned int *>(e->arena.get("q18.counts", 4ull * 256 * sort_tiles(nout)));
         sp2.totals = static_cast<unsigned int *>(e->arena.get("q18.totals", 4 * 256));
+        BucketSort bs;
+        bs.k[0] = sp2.k[0]; bs.k[1] = sp2.k[1]; bs.v[0] = sp2.v[0]; bs.v[1] = sp2.v[1];
+        bs.count = static_cast<unsigned int *>(e->arena.get("q18.bcount", 4 * (8192 + 1)));
+        bs.cursor = static_cast<unsigned int *>(e->arena.get("q18.bcursor", 4 * 8192));
+        bs.offset = static_cast<unsigned int *>(e->arena.get("q18.boffset", 4 * (8192 + 1)));
+        int bb = 1;
+        while (bb < 13 && (nout >> (bb + 9)) > 0) ++bb;   // ~512 rows per bucket on average
         e->prof.run("q18_sort_keys", [&] { launch_q18_sort_keys(rows, nout, sp, sp2, e->num_sms, e->compute); });
-        int cur = 0;
-        e->prof.run("q18_radix_sort", [&] { cur = radix_sort_pairs(nout, sp.prefix_bits, sp2, e->num_sms, e->compute); });
-        perm = sp2.v[cur];
-        if (tiefix) {
-            CK(cudaMemsetAsync(tie_dev, 0, 4, e->compute));
+        CK(cudaMemsetAsync(tie_dev, 0, 4, e->compute));
+        e->prof.run("q18_bucket_sort", [&] {
+            bucket_sort_pairs(nout, sp.prefix_bits, bb, bs, tie_dev, e->num_sms, e->compute);
+        });
+        perm = sp2.v[1];
+        if (tiefix)
             e->prof.run("q18_tiefix", [&] {
-                launch_q18_tiefix(rows, sp2.k[cur], sp2.v[cur], nout, tie_dev, e->num_sms, e->compute);
+                launch_q18_tiefix(rows, sp2.k[1], sp2.v[1], nout, tie_dev, e->num_sms, e->compute);
             });
-        }
+        tiefix = true;  // read the flag back: tie runs > 32 (bit 0) or a bucket > capacity (bit 1)
     }
     r->nrows = nout;
     Q18Cols dst;
@@ -902,7 +910,8 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
     };
     emit();
     if (tiefix && sm->tie) {
-        // a run of > 32 equal prefixes: redo exactly, one stable LSD sort per field (r, e, a)
+        // a run of > 32 equal 64-bit prefixes, or a bucket larger than shared memory: redo
+        // exactly, one stable LSD radix sort per field (r, then e, then a)
         SortPairs w = sp2;
         launch_iota(w.v[0], nout, e->num_sms, e->compute);
         const int fb[3] = {sp.bits_r, sp.bits_e, sp.bits_a};

@@ -229,51 +229,79 @@ struct StatAcc {
     }
 };
 
+// Each block iteration covers kHavingRows consecutive orders rows (kHavingUnroll per thread);
+// passing rows get output slots from ONE atomicAdd per block iteration (block-wide exclusive
+// scan of the per-thread counts), so the output counter sees ~n/1024 atomics, not n/32.
+constexpr int kHavingUnroll = 4;
+constexpr int kHavingRows = kHavingThreads * kHavingUnroll;
+
 __global__ void __launch_bounds__(kHavingThreads)
 q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
                   const int32_t *__restrict__ o_id, const int32_t *__restrict__ o_c,
                   const int32_t *__restrict__ o_cnt, const int64_t *__restrict__ o_ent, uint64_t n,
                   const int32_t *__restrict__ c_last, long long having, Q18Scratch s) {
-    const int lane = threadIdx.x & 31;
-    const uint64_t gwarp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
-    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
+    __shared__ unsigned int wsum[kHavingThreads / 32];
+    __shared__ unsigned long long s_base;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     StatAcc stat;
-    for (uint64_t base = gwarp * 32; base < n; base += nwarps * 32) {
-        const uint64_t r = base + lane;
-        bool pass = false;
-        unsigned int crow = kNoRow;
-        long long sum = 0;
-        int w = 0, d = 0, c = 0;
-        if (r < n) {
-            const ulonglong2 a = __ldcs(reinterpret_cast<const ulonglong2 *>(s.acc + r));
-            sum = (long long)a.x;
-            const unsigned int cnt = (unsigned int)a.y;
-            // inner join: a group exists only with >= 1 order_line row; HAVING SUM > having
-            if (cnt > 0 && sum > having) {
-                w = o_w[r]; d = o_d[r]; c = o_c[r];
-                crow = jx_lookup(s.jc, w, d, c);  // customer ⋈ orders
-                pass = crow != kNoRow;
+    for (uint64_t base = (uint64_t)blockIdx.x * kHavingRows; base < n;
+         base += (uint64_t)gridDim.x * kHavingRows) {
+        unsigned int crow[kHavingUnroll];
+        long long sum[kHavingUnroll];
+        int w[kHavingUnroll], d[kHavingUnroll], c[kHavingUnroll];
+        unsigned int mine = 0;
+#pragma unroll
+        for (int u = 0; u < kHavingUnroll; ++u) {
+            const uint64_t r = base + u * kHavingThreads + threadIdx.x;
+            crow[u] = kNoRow;
+            sum[u] = 0;
+            w[u] = d[u] = c[u] = 0;
+            if (r < n) {
+                const ulonglong2 a = __ldcs(reinterpret_cast<const ulonglong2 *>(s.acc + r));
+                sum[u] = (long long)a.x;
+                // inner join: a group exists only with >= 1 order_line row; HAVING SUM > having
+                if ((unsigned int)a.y > 0 && sum[u] > having) {
+                    w[u] = o_w[r]; d[u] = o_d[r]; c[u] = o_c[r];
+                    crow[u] = jx_lookup(s.jc, w[u], d[u], c[u]);  // customer ⋈ orders
+                }
             }
+            mine += crow[u] != kNoRow;
         }
-        const unsigned ball = __ballot_sync(kFull, pass);
-        if (!ball) continue;
-        unsigned long long basepos = 0;
-        if (lane == 0) basepos = atomicAdd(s.nout, (unsigned long long)__popc(ball));
-        basepos = __shfl_sync(kFull, basepos, 0);
-        if (pass) {
-            const uint64_t p = basepos + __popc(ball & ((1u << lane) - 1u));
+        // block-wide exclusive scan of `mine`, one atomic for the block's output range
+        unsigned int x = mine;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const unsigned int t = __shfl_up_sync(kFull, x, o);
+            if (lane >= o) x += t;
+        }
+        if (lane == 31) wsum[warp] = x;
+        __syncthreads();
+        unsigned int before = 0, total = 0;
+#pragma unroll
+        for (int k = 0; k < kHavingThreads / 32; ++k) {
+            before += k < warp ? wsum[k] : 0u;
+            total += wsum[k];
+        }
+        if (threadIdx.x == 0) s_base = total ? atomicAdd(s.nout, (unsigned long long)total) : 0ull;
+        __syncthreads();
+        uint64_t p = s_base + before + x - mine;
+#pragma unroll
+        for (int u = 0; u < kHavingUnroll; ++u) {
+            if (crow[u] == kNoRow) continue;
+            const uint64_t r = base + u * kHavingThreads + threadIdx.x;
             Q18Row row;
-            row.amount_sum = sum;
+            row.amount_sum = sum[u];
             row.o_entry_d = o_ent[r];
-            row.c_last = c_last[crow];
-            row.c_id = c;
+            row.c_last = c_last[crow[u]];
+            row.c_id = c[u];
             row.o_id = o_id[r];
             row.o_ol_cnt = o_cnt[r];
-            row.o_w_id = w;
-            row.o_d_id = d;
-            s.rows[p] = row;
-            stat.add(sum, row.o_entry_d, w, d, row.o_id);
+            row.o_w_id = w[u];
+            row.o_d_id = d[u];
+            s.rows[p++] = row;
+            stat.add(sum[u], row.o_entry_d, w[u], d[u], row.o_id);
         }
+        __syncthreads();  // wsum / s_base reuse
     }
     stat.flush(s.stats);
 }
@@ -316,7 +344,8 @@ void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_
                        const int32_t *o_c, const int32_t *o_cnt, const int64_t *o_ent,
                        uint64_t n_o, const int32_t *c_last, int64_t having,
                        const Q18Scratch &s, int num_sms, cudaStream_t st) {
-    q18_having_kernel<<<grid_for(n_o, kHavingThreads, num_sms, 8), kHavingThreads, 0, st>>>(
+    q18_having_kernel<<<grid_for((n_o + kHavingUnroll - 1) / kHavingUnroll, kHavingThreads, num_sms, 8),
+                        kHavingThreads, 0, st>>>(
         o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o, c_last, having, s);
     count_launches(1);
 }

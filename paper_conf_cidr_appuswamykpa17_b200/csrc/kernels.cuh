@@ -117,6 +117,21 @@ struct SortPairs {
 // Returns which buffer (0/1) holds the sorted pairs (input is in k[0]/v[0]).
 int radix_sort_pairs(uint64_t n, int bits, const SortPairs &s, int num_sms, cudaStream_t st);
 
+// Bucket sort of (u64 key, u32 value) pairs whose keys use the low `bits` bits: partition by the
+// top `bucket_bits` key bits (histogram -> scan -> scatter), then sort every bucket in shared
+// memory (bitonic). A bucket larger than kBucketCap raises *flag (caller falls back to LSD).
+constexpr int kBucketCap = 8192;
+struct BucketSort {
+    unsigned long long *k[2];
+    unsigned int *v[2];
+    unsigned int *count;   // [2^bucket_bits + 1]
+    unsigned int *cursor;  // [2^bucket_bits]
+    unsigned int *offset;  // [2^bucket_bits + 1]
+};
+// Sorted pairs end in k[1]/v[1] (input in k[0]/v[0]).
+void bucket_sort_pairs(uint64_t n, int bits, int bucket_bits, const BucketSort &s, unsigned int *flag,
+                       int num_sms, cudaStream_t st);
+
 // Q18 ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id (R11).
 struct Q18SortSpec {         // host-computed from Q18Stats
     long long amt_max, ent_min;

@@ -4,12 +4,13 @@
 // The three sort fields are mapped to unsigned integers whose widths come from the result's
 // min/max (HAVING kernel statistics): a = max - amount_sum (DESC), e = o_entry_d - min,
 // r = dense rank of (w, d, o). Their concatenation a|e|r is the exact composite key.
-//  * composite <= 64 bits: one stable LSD radix sort of (key, row) pairs — exact.
-//  * wider: sort by the composite's top `prefix_bits`, then order each run of equal prefixes by
-//    the full tuple (runs are a handful of rows on realistic data); a run longer than 32 rows
-//    raises a flag and the engine redoes the sort exactly, field by field (r, then e, then a).
-// Radix pass = per-tile digit histogram -> per-digit scan -> stable scatter; keys travel with
-// their row ids so every pass reads and writes contiguous arrays.
+//  * main path: sort (top 64 bits of a|e|r, row id) pairs with a bucket sort (partition by the
+//    top key bits, bitonic sort per bucket in shared memory). If a|e|r fits 64 bits the keys are
+//    distinct and the order is exact; otherwise runs of equal 64-bit prefixes are ordered by the
+//    full tuple (tie-fix; runs are a handful of rows on realistic data).
+//  * exact fallback (a run > 32 rows or a bucket > shared memory): one stable LSD radix sort of
+//    (key, row) pairs per field, r then e then a. Radix pass = per-tile digit histogram ->
+//    per-digit scan -> stable scatter; keys travel with their row ids.
 #include <cstdint>
 #include <cuda_runtime.h>
 
@@ -313,6 +314,180 @@ void launch_iota(unsigned int *v, uint64_t n, int num_sms, cudaStream_t st) {
 void launch_q18_permute(const Q18Row *rows, const unsigned int *perm, uint64_t n,
                         const Q18Cols &dst, int num_sms, cudaStream_t st) {
     permute_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, perm, n, dst);
+    count_launches(1);
+}
+
+}  // namespace h2tap
+
+// ============================================================ bucket sort ===
+// Main ORDER BY path: the result (a few million 12-byte pairs) fits in L2, so
+// one partition pass by the top key bits plus a shared-memory sort per bucket replaces the
+// 6 LSD passes. Buckets are not stable internally; equal full prefixes are ordered afterwards by
+// the tie-fix kernel (which sorts runs of equal prefix by the full tuple) — so the result is the
+// same total order as the LSD path.
+namespace h2tap {
+namespace {
+
+constexpr int kBkThreads = 256;
+constexpr int kBkSmemBins = 8192;  // max buckets counted in shared memory per block
+
+__global__ void __launch_bounds__(kBkThreads)
+bucket_hist_kernel(const unsigned long long *__restrict__ key, uint64_t n, int shift, int nb,
+                   unsigned int *__restrict__ count) {
+    extern __shared__ unsigned int h[];
+    for (int i = threadIdx.x; i < nb; i += kBkThreads) h[i] = 0;
+    __syncthreads();
+    const uint64_t stride = (uint64_t)gridDim.x * kBkThreads;
+    for (uint64_t i = (uint64_t)blockIdx.x * kBkThreads + threadIdx.x; i < n; i += stride)
+        atomicAdd(&h[(unsigned int)(__ldcg(key + i) >> shift)], 1u);
+    __syncthreads();
+    for (int i = threadIdx.x; i < nb; i += kBkThreads)
+        if (h[i]) atomicAdd(count + i, h[i]);
+}
+
+// exclusive scan of nb bucket counts -> offset[] and cursor[]; max bucket size -> count[nb]
+__global__ void __launch_bounds__(1024) bucket_scan_kernel(unsigned int *__restrict__ count, int nb,
+                                                           unsigned int *__restrict__ offset,
+                                                           unsigned int *__restrict__ cursor) {
+    __shared__ unsigned int wsum[32];
+    __shared__ unsigned int carry_s;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    unsigned int carry = 0, mx = 0;
+    for (int r0 = 0; r0 < nb; r0 += 1024) {
+        const int i = r0 + threadIdx.x;
+        const unsigned int v = i < nb ? count[i] : 0u;
+        mx = max(mx, v);
+        unsigned int x = v;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const unsigned int t = __shfl_up_sync(kFull, x, o);
+            if (lane >= o) x += t;
+        }
+        if (lane == 31) wsum[warp] = x;
+        __syncthreads();
+        if (warp == 0) {
+            unsigned int y = wsum[lane];
+#pragma unroll
+            for (int o = 1; o < 32; o <<= 1) {
+                const unsigned int t = __shfl_up_sync(kFull, y, o);
+                if (lane >= o) y += t;
+            }
+            wsum[lane] = y;
+            if (lane == 31) carry_s = y;
+        }
+        __syncthreads();
+        const unsigned int ex = carry + (warp ? wsum[warp - 1] : 0u) + x - v;
+        if (i < nb) { offset[i] = ex; cursor[i] = ex; }
+        carry += carry_s;
+        __syncthreads();
+    }
+    mx = __reduce_max_sync(kFull, mx);
+    if (lane == 0) wsum[warp] = mx;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        unsigned int m = 0;
+        for (int w = 0; w < 32; ++w) m = max(m, wsum[w]);
+        offset[nb] = carry;
+        count[nb] = m;
+    }
+}
+
+// scatter into buckets: per-block shared histogram reserves one global range per bucket
+__global__ void __launch_bounds__(kBkThreads)
+bucket_scatter_kernel(const unsigned long long *__restrict__ kin, const unsigned int *__restrict__ vin,
+                      unsigned long long *__restrict__ kout, unsigned int *__restrict__ vout, uint64_t n,
+                      int shift, int nb, unsigned int *__restrict__ cursor, uint64_t per_block) {
+    extern __shared__ unsigned int h[];  // [nb] local counts -> local cursors
+    for (int i = threadIdx.x; i < nb; i += kBkThreads) h[i] = 0;
+    __syncthreads();
+    const uint64_t lo = (uint64_t)blockIdx.x * per_block;
+    const uint64_t hi = lo + per_block < n ? lo + per_block : n;
+    for (uint64_t i = lo + threadIdx.x; i < hi; i += kBkThreads)
+        atomicAdd(&h[(unsigned int)(__ldcg(kin + i) >> shift)], 1u);
+    __syncthreads();
+    for (int i = threadIdx.x; i < nb; i += kBkThreads)
+        if (h[i]) h[i] = atomicAdd(cursor + i, h[i]);  // base of this block's range in bucket i
+    __syncthreads();
+    for (uint64_t i = lo + threadIdx.x; i < hi; i += kBkThreads) {
+        const unsigned long long k = __ldcg(kin + i);
+        const unsigned int p = atomicAdd(&h[(unsigned int)(k >> shift)], 1u);
+        kout[p] = k;
+        vout[p] = __ldcg(vin + i);
+    }
+}
+
+// one block per bucket: load into shared memory, bitonic sort by key, write back
+__global__ void __launch_bounds__(kBkThreads)
+bucket_local_sort_kernel(unsigned long long *__restrict__ k, unsigned int *__restrict__ v,
+                         const unsigned int *__restrict__ offset, int nb, unsigned int *flag) {
+    extern __shared__ unsigned long long sk[];  // [kBucketCap] keys, then [kBucketCap] values
+    unsigned int *sv = reinterpret_cast<unsigned int *>(sk + kBucketCap);
+    for (int b = blockIdx.x; b < nb; b += gridDim.x) {
+        const unsigned int lo = offset[b], cnt = offset[b + 1] - lo;
+        if (cnt <= 1) continue;
+        if (cnt > (unsigned)kBucketCap) {
+            if (threadIdx.x == 0) atomicOr(flag, 2u);
+            continue;
+        }
+        unsigned int m = 2;
+        while (m < cnt) m <<= 1;
+        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
+            sk[i] = i < cnt ? k[lo + i] : ~0ull;
+            sv[i] = i < cnt ? v[lo + i] : 0u;
+        }
+        __syncthreads();
+        for (unsigned int size = 2; size <= m; size <<= 1) {
+            for (unsigned int stride = size >> 1; stride > 0; stride >>= 1) {
+                for (unsigned int t = threadIdx.x; t < m / 2; t += kBkThreads) {
+                    const unsigned int i = 2 * t - (t & (stride - 1));
+                    const unsigned int j = i + stride;
+                    const bool up = (i & size) == 0;
+                    const unsigned long long a = sk[i], c = sk[j];
+                    if ((a > c) == up) {
+                        sk[i] = c; sk[j] = a;
+                        const unsigned int tv = sv[i]; sv[i] = sv[j]; sv[j] = tv;
+                    }
+                }
+                __syncthreads();
+            }
+        }
+        for (unsigned int i = threadIdx.x; i < cnt; i += kBkThreads) {
+            k[lo + i] = sk[i];
+            v[lo + i] = sv[i];
+        }
+        __syncthreads();
+    }
+}
+
+}  // namespace
+
+void bucket_sort_pairs(uint64_t n, int bits, int bucket_bits, const BucketSort &s, unsigned int *flag,
+                       int num_sms, cudaStream_t st) {
+    if (bucket_bits > bits) bucket_bits = bits;
+    if (bucket_bits > 13) bucket_bits = 13;  // shared histogram of <= 8192 bins
+    const int nb = 1 << bucket_bits;
+    const int shift = bits - bucket_bits;
+    static bool init = false;
+    if (!init) {
+        cudaFuncSetAttribute(bucket_local_sort_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             kBucketCap * 12);
+        init = true;
+    }
+    cudaMemsetAsync(s.count, 0, sizeof(unsigned int) * (nb + 1), st);
+    uint64_t hb = (n + kBkThreads * 16 - 1) / (kBkThreads * 16);
+    if (hb > (uint64_t)num_sms * 4) hb = (uint64_t)num_sms * 4;
+    if (!hb) hb = 1;
+    bucket_hist_kernel<<<(unsigned)hb, kBkThreads, nb * 4, st>>>(s.k[0], n, shift, nb, s.count);
+    count_launches(1);
+    bucket_scan_kernel<<<1, 1024, 0, st>>>(s.count, nb, s.offset, s.cursor);
+    count_launches(1);
+    const uint64_t per_block = 16384;
+    const uint64_t sb = (n + per_block - 1) / per_block;
+    bucket_scatter_kernel<<<(unsigned)(sb ? sb : 1), kBkThreads, nb * 4, st>>>(
+        s.k[0], s.v[0], s.k[1], s.v[1], n, shift, nb, s.cursor, per_block);
+    count_launches(1);
+    unsigned lb = (unsigned)nb < (unsigned)num_sms * 16 ? (unsigned)nb : (unsigned)num_sms * 16;
+    bucket_local_sort_kernel<<<lb, kBkThreads, kBucketCap * 12, st>>>(s.k[1], s.v[1], s.offset, nb, flag);
     count_launches(1);
 }
 
