@@ -725,7 +725,10 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
     s.err = static_cast<unsigned int *>(e->arena.get("q18.err", 64));
     s.nout = static_cast<unsigned long long *>(e->arena.get("q18.nout", 64));
     s.stats = static_cast<Q18Stats *>(e->arena.get("q18.stats", sizeof(Q18Stats)));
+    s.stat_part = static_cast<Q18Stats *>(e->arena.get("q18.statpart", sizeof(Q18Stats) * 8 * e->num_sms));
+    s.ticket = static_cast<unsigned int *>(e->arena.get("q18.ticket", 64, true, e->compute));
     s.rows = static_cast<Q18Row *>(e->arena.get("q18.rows", sizeof(Q18Row) * std::max<uint64_t>(n_o, 1)));
+    s.amt = static_cast<long long *>(e->arena.get("q18.amt", 8 * std::max<uint64_t>(n_o, 1)));
     r->plan_flags = (s.jo.dense ? 1u : 0u) | (s.jc.dense ? 2u : 0u);
 
     e->prof.run("q18_init", [&] { launch_q18_init(s, n_o, e->num_sms, e->compute); });
@@ -774,6 +777,7 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
     if (err_any) raise(H2TAP_EPLAN, "Q18: failed on another rank");
 
     const Q18Row *rows = s.rows;
+    const long long *amt = s.amt;
     if (e->world > 1) {  // a7: groups are warehouse-local; gather result rows to rank 0
         auto *cnt_dev = static_cast<unsigned long long *>(e->arena.get("q18.allcnt", 8ull * e->world));
         NK(ncclAllGather(s.nout, cnt_dev, 1, ncclUint64, e->comm, e->compute));
@@ -784,18 +788,24 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
         for (auto c : cnts) total += c;
         Q18Row *all = e->rank == 0 ? static_cast<Q18Row *>(e->arena.get("q18.allrows", sizeof(Q18Row) * std::max<uint64_t>(total, 1)))
                                    : nullptr;
+        long long *all_amt = e->rank == 0 ? static_cast<long long *>(e->arena.get("q18.allamt", 8 * std::max<uint64_t>(total, 1)))
+                                          : nullptr;
         e->prof.run("q18_gather", [&] {
             NK(ncclGroupStart());
             uint64_t off = 0;
             for (int k = 0; k < e->world; ++k) {
-                const size_t bytes = cnts[k] * sizeof(Q18Row);
+                const size_t bytes = cnts[k] * sizeof(Q18Row), abytes = cnts[k] * 8;
                 if (bytes) {
-                    if (e->rank == 0 && k == 0)
+                    if (e->rank == 0 && k == 0) {
                         CK(cudaMemcpyAsync(all, s.rows, bytes, cudaMemcpyDeviceToDevice, e->compute));
-                    else if (e->rank == 0)
+                        CK(cudaMemcpyAsync(all_amt, s.amt, abytes, cudaMemcpyDeviceToDevice, e->compute));
+                    } else if (e->rank == 0) {
                         NK(ncclRecv(all + off, bytes, ncclUint8, k, e->comm, e->compute));
-                    else if (e->rank == k)
+                        NK(ncclRecv(all_amt + off, abytes, ncclUint8, k, e->comm, e->compute));
+                    } else if (e->rank == k) {
                         NK(ncclSend(s.rows, bytes, ncclUint8, 0, e->comm, e->compute));
+                        NK(ncclSend(s.amt, abytes, ncclUint8, 0, e->comm, e->compute));
+                    }
                 }
                 off += cnts[k];
             }
@@ -812,13 +822,14 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
         }
         nout = total;
         rows = all;
+        amt = all_amt;
         Q18Stats init;
         init.amt_min = INT64_MAX; init.amt_max = INT64_MIN; init.ent_min = INT64_MAX; init.ent_max = INT64_MIN;
         init.w_min = INT32_MAX; init.w_max = INT32_MIN; init.d_min = INT32_MAX; init.d_max = INT32_MIN;
         init.o_min = INT32_MAX; init.o_max = INT32_MIN; init.pad0 = init.pad1 = 0;
         sm->st = init;
         CK(cudaMemcpyAsync(s.stats, &sm->st, sizeof(Q18Stats), cudaMemcpyHostToDevice, e->compute));
-        launch_q18_stats(rows, nout, s.stats, e->num_sms, e->compute);
+        launch_q18_stats(rows, amt, nout, s, e->num_sms, e->compute);
         CK(cudaMemcpyAsync(&sm->st, s.stats, sizeof(Q18Stats), cudaMemcpyDeviceToHost, e->compute));
         sync_compute(e);
         st = sm->st;
@@ -828,6 +839,7 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
     Q18SortSpec sp{};
     SortPairs sp2{};
     const unsigned int *perm = nullptr;
+    const unsigned long long *perm_keys = nullptr;  // sorted prefix keys parallel to perm
     unsigned int *tie_dev = static_cast<unsigned int *>(e->arena.get("q18.tie", 64));
     bool tiefix = false;
     if (nout > 1) {
@@ -851,20 +863,21 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
         sp2.totals = static_cast<unsigned int *>(e->arena.get("q18.totals", 4 * 256));
         BucketSort bs;
         bs.k[0] = sp2.k[0]; bs.k[1] = sp2.k[1]; bs.v[0] = sp2.v[0]; bs.v[1] = sp2.v[1];
-        bs.count = static_cast<unsigned int *>(e->arena.get("q18.bcount", 4 * (8192 + 1)));
-        bs.cursor = static_cast<unsigned int *>(e->arena.get("q18.bcursor", 4 * 8192));
-        bs.offset = static_cast<unsigned int *>(e->arena.get("q18.boffset", 4 * (8192 + 1)));
+        bs.count = static_cast<unsigned int *>(e->arena.get("q18.bcount", 4 * ((1 << kBucketMaxBits) + 1)));
+        bs.cursor = static_cast<unsigned int *>(e->arena.get("q18.bcursor", 4 * (1 << kBucketMaxBits)));
+        bs.offset = static_cast<unsigned int *>(e->arena.get("q18.boffset", 4 * ((1 << kBucketMaxBits) + 1)));
         int bb = 1;
-        while (bb < 13 && (nout >> (bb + 9)) > 0) ++bb;   // ~512 rows per bucket on average
-        e->prof.run("q18_sort_keys", [&] { launch_q18_sort_keys(rows, nout, sp, sp2, e->num_sms, e->compute); });
+        while (bb < kBucketMaxBits && (nout >> (bb + 9)) > 0) ++bb;   // ~256-512 rows per bucket
+        e->prof.run("q18_sort_keys", [&] { launch_q18_sort_keys(rows, amt, nout, sp, sp2, e->num_sms, e->compute); });
         CK(cudaMemsetAsync(tie_dev, 0, 4, e->compute));
         e->prof.run("q18_bucket_sort", [&] {
             bucket_sort_pairs(nout, sp.prefix_bits, bb, bs, tie_dev, e->num_sms, e->compute);
         });
         perm = sp2.v[1];
+        perm_keys = sp2.k[1];
         if (tiefix)
             e->prof.run("q18_tiefix", [&] {
-                launch_q18_tiefix(rows, sp2.k[1], sp2.v[1], nout, tie_dev, e->num_sms, e->compute);
+                launch_q18_tiefix(rows, amt, sp2.k[1], sp2.v[1], nout, tie_dev, e->num_sms, e->compute);
             });
         tiefix = true;  // read the flag back: tie runs > 32 (bit 0) or a bucket > capacity (bit 1)
     }
@@ -893,7 +906,9 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
         host_dst.o_d_id = static_cast<int32_t *>(result_block(r, 4 * nout));
     }
     auto emit = [&]() {
-        e->prof.run("q18_permute", [&] { if (nout) launch_q18_permute(rows, perm, nout, dst, e->num_sms, e->compute); });
+        e->prof.run("q18_permute", [&] {
+            if (nout) launch_q18_permute(rows, amt, perm, perm_keys, sp, nout, dst, e->num_sms, e->compute);
+        });
         if (!r->on_device && nout) {
             auto d2h = [&](void *h, const void *d, size_t es) {
                 CK(cudaMemcpyAsync(h, d, nout * es, cudaMemcpyDeviceToHost, e->compute));
@@ -916,11 +931,12 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
         launch_iota(w.v[0], nout, e->num_sms, e->compute);
         const int fb[3] = {sp.bits_r, sp.bits_e, sp.bits_a};
         for (int f = 0; f < 3; ++f) {
-            launch_q18_field_keys(rows, w.v[0], nout, f, sp, w.k[0], e->num_sms, e->compute);
+            launch_q18_field_keys(rows, amt, w.v[0], nout, f, sp, w.k[0], e->num_sms, e->compute);
             const int cur = radix_sort_pairs(nout, fb[f], w, e->num_sms, e->compute);
             if (cur) { std::swap(w.k[0], w.k[1]); std::swap(w.v[0], w.v[1]); }
         }
         perm = w.v[0];
+        perm_keys = nullptr;  // field keys, not the prefix: amounts are read from amt[]
         tiefix = false;
         emit();
     }

@@ -134,12 +134,26 @@ __global__ void q18_build_kernel(const int32_t *__restrict__ o_w, const int32_t 
 }
 
 // ------------------------------------------------------- K4 probe + group-join --
-// One warp iteration covers 32 consecutive order_line rows (coalesced 4 B / 8 B loads).
-// Lines of one order are usually contiguous, so equal keys form runs: a segmented inclusive
-// scan (shuffles) sums each run, the run head probes the orders index once, and the run tail
-// issues the two atomics — ~3 runs per 32 rows instead of 32 probes and 64 atomics.
+// Each lane owns 4 consecutive order_line rows (128-bit loads of w, d, o and two of amount), so
+// a warp iteration covers 128 rows. Lines of one order are contiguous, so equal (w, d, o) keys
+// form runs (~10 rows): runs are summed inside the lane, a run crossing lanes is summed by a
+// 5-step segmented shuffle scan over the lanes' last partial runs, and each run issues ONE
+// probe of the orders index and two atomics into acc[orders row] from the lane where it ends.
 constexpr int kProbeThreads = 256;
-constexpr int kProbeUnroll = 4;
+
+struct Key3 { int w, d, o; };
+__device__ __forceinline__ bool eq3(const Key3 &a, const Key3 &b) {
+    return (a.w == b.w) & (a.d == b.d) & (a.o == b.o);
+}
+
+__device__ __forceinline__ void flush_run(const Q18Scratch &s, const Key3 &k, long long sum,
+                                          unsigned int cnt) {
+    const unsigned int row = jx_lookup(s.jo, k.w, k.d, k.o);
+    if (row != kNoRow) {
+        atomicAdd(reinterpret_cast<unsigned long long *>(&s.acc[row].sum), (unsigned long long)sum);
+        atomicAdd(&s.acc[row].cnt, cnt);
+    }
+}
 
 __global__ void __launch_bounds__(kProbeThreads)
 q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ ol_d,
@@ -148,47 +162,63 @@ q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ o
     const int lane = threadIdx.x & 31;
     const uint64_t gwarp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
-    const unsigned le_mask = 0xffffffffu >> (31 - lane);  // lanes 0..lane
-    for (uint64_t base = gwarp * 32 * kProbeUnroll; base < n; base += nwarps * 32 * kProbeUnroll) {
-        int w[kProbeUnroll], d[kProbeUnroll], o[kProbeUnroll];
-        long long amt[kProbeUnroll];
-        bool valid[kProbeUnroll];
-#pragma unroll
-        for (int u = 0; u < kProbeUnroll; ++u) {
-            const uint64_t i = base + u * 32 + lane;
-            valid[u] = i < n;
-            if (valid[u]) {
-                w[u] = __ldcs(ol_w + i); d[u] = __ldcs(ol_d + i); o[u] = __ldcs(ol_o + i);
-                amt[u] = __ldcs(ol_amt + i);
-            } else {  // tail rows: never probe, never aggregate
-                w[u] = 0; d[u] = 0; o[u] = 0; amt[u] = 0;
-            }
+    const uint64_t nvec = n >> 2;  // full 4-row groups; the ragged tail is handled below
+    for (uint64_t vb = gwarp * 32; vb < nvec; vb += nwarps * 32) {
+        const uint64_t v = vb + lane;
+        const bool valid = v < nvec;
+        Key3 k[4];
+        long long a[4];
+        if (valid) {
+            const int4 W = __ldcs(reinterpret_cast<const int4 *>(ol_w) + v);
+            const int4 D = __ldcs(reinterpret_cast<const int4 *>(ol_d) + v);
+            const int4 O = __ldcs(reinterpret_cast<const int4 *>(ol_o) + v);
+            const longlong2 A0 = __ldcs(reinterpret_cast<const longlong2 *>(ol_amt) + 2 * v);
+            const longlong2 A1 = __ldcs(reinterpret_cast<const longlong2 *>(ol_amt) + 2 * v + 1);
+            k[0] = {W.x, D.x, O.x}; k[1] = {W.y, D.y, O.y}; k[2] = {W.z, D.z, O.z}; k[3] = {W.w, D.w, O.w};
+            a[0] = A0.x; a[1] = A0.y; a[2] = A1.x; a[3] = A1.y;
+        } else {
+            for (int j = 0; j < 4; ++j) { k[j] = {0, 0, 0}; a[j] = 0; }
         }
+        // in-lane runs: b[j] = row j starts a run; s[j], c[j] = running sum / count of its run
+        bool b1 = !eq3(k[1], k[0]), b2 = !eq3(k[2], k[1]), b3 = !eq3(k[3], k[2]);
+        long long s0 = a[0], s1 = (b1 ? 0 : s0) + a[1], s2 = (b2 ? 0 : s1) + a[2], s3 = (b3 ? 0 : s2) + a[3];
+        unsigned c0 = 1, c1 = (b1 ? 0 : c0) + 1, c2 = (b2 ? 0 : c1) + 1, c3 = (b3 ? 0 : c2) + 1;
+        const bool multi = b1 | b2 | b3;
+        // does my first run continue the previous lane's last run?
+        const int pw = __shfl_up_sync(kFull, k[3].w, 1), pd = __shfl_up_sync(kFull, k[3].d, 1),
+                  po = __shfl_up_sync(kFull, k[3].o, 1);
+        const bool pvalid = __shfl_up_sync(kFull, valid, 1);
+        const bool cont = lane > 0 && valid && pvalid && pw == k[0].w && pd == k[0].d && po == k[0].o;
+        const bool next_cont = __shfl_down_sync(kFull, cont, 1) && lane < 31;
+        // segmented inclusive scan of the lanes' last partial runs (segment starts where a lane
+        // does not continue, or where its last run starts inside the lane)
+        const bool start = !cont || multi;
+        const unsigned starts = __ballot_sync(kFull, start);
+        const int seg = 31 - __clz(starts & (0xffffffffu >> (31 - lane)));
+        long long is = s3;
+        unsigned ic = c3;
 #pragma unroll
-        for (int u = 0; u < kProbeUnroll; ++u) {
-            const bool same = (__shfl_up_sync(kFull, w[u], 1) == w[u]) &
-                              (__shfl_up_sync(kFull, d[u], 1) == d[u]) &
-                              (__shfl_up_sync(kFull, o[u], 1) == o[u]) &
-                              (__shfl_up_sync(kFull, (int)valid[u], 1) == (int)valid[u]);
-            const bool head = lane == 0 || !same;
-            const unsigned heads = __ballot_sync(kFull, head);
-            const int leader = 31 - __clz(heads & le_mask);
-            long long sum = amt[u];
-#pragma unroll
-            for (int off = 1; off < 32; off <<= 1) {
-                const long long t = __shfl_up_sync(kFull, sum, off);
-                if (lane - off >= leader) sum += t;
-            }
-            const bool tail = lane == 31 || ((heads >> (lane + 1)) & 1u);
-            unsigned int row = kNoRow;
-            if (head && valid[u]) row = jx_lookup(s.jo, w[u], d[u], o[u]);
-            row = __shfl_sync(kFull, row, leader);
-            if (tail && row != kNoRow) {
-                atomicAdd(reinterpret_cast<unsigned long long *>(&s.acc[row].sum),
-                          (unsigned long long)sum);
-                atomicAdd(&s.acc[row].cnt, (unsigned int)(lane - leader + 1));
-            }
+        for (int off = 1; off < 32; off <<= 1) {
+            const long long ts = __shfl_up_sync(kFull, is, off);
+            const unsigned tc = __shfl_up_sync(kFull, ic, off);
+            if (lane - off >= seg) { is += ts; ic += tc; }
         }
+        // carry into my first run = inclusive value of the previous lane (if I continue it)
+        long long carry_s = __shfl_up_sync(kFull, is, 1);
+        unsigned carry_c = __shfl_up_sync(kFull, ic, 1);
+        if (!cont) { carry_s = 0; carry_c = 0; }
+        if (!valid) continue;
+        // runs ending inside the lane (rows 0..2): the first run also gets the carry
+        if (b1) flush_run(s, k[0], s0 + carry_s, c0 + carry_c);
+        if (b2) flush_run(s, k[1], s1 + (b1 ? 0 : carry_s), c1 + (b1 ? 0 : carry_c));
+        if (b3) flush_run(s, k[2], s2 + ((b1 | b2) ? 0 : carry_s), c2 + ((b1 | b2) ? 0 : carry_c));
+        // the lane's last run ends here unless the next lane continues it
+        if (!next_cont) flush_run(s, k[3], is, ic);
+    }
+    // ragged tail (< 4 rows) plus nothing else: one thread, row at a time
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
+        for (uint64_t i = nvec * 4; i < n; ++i)
+            flush_run(s, Key3{ol_w[i], ol_d[i], ol_o[i]}, ol_amt[i], 1u);
     }
 }
 
@@ -214,17 +244,61 @@ struct StatAcc {
         wmin = min(wmin, w); wmax = max(wmax, w); dmin = min(dmin, d); dmax = max(dmax, d);
         omin = min(omin, o); omax = max(omax, o);
     }
-    __device__ void flush(Q18Stats *st) {  // warp-reduce, lane 0 issues the atomics
+    __device__ void merge(const Q18Stats &o) {
+        amin = o.amt_min < amin ? o.amt_min : amin; amax = o.amt_max > amax ? o.amt_max : amax;
+        emin = o.ent_min < emin ? o.ent_min : emin; emax = o.ent_max > emax ? o.ent_max : emax;
+        wmin = min(wmin, o.w_min); wmax = max(wmax, o.w_max); dmin = min(dmin, o.d_min);
+        dmax = max(dmax, o.d_max); omin = min(omin, o.o_min); omax = max(omax, o.o_max);
+    }
+    __device__ void warp_reduce() {
         amin = wmin64(amin); amax = wmax64(amax); emin = wmin64(emin); emax = wmax64(emax);
         wmin = __reduce_min_sync(kFull, wmin); wmax = __reduce_max_sync(kFull, wmax);
         dmin = __reduce_min_sync(kFull, dmin); dmax = __reduce_max_sync(kFull, dmax);
         omin = __reduce_min_sync(kFull, omin); omax = __reduce_max_sync(kFull, omax);
-        if ((threadIdx.x & 31) == 0 && amin <= amax) {
-            atomicMin(&st->amt_min, amin); atomicMax(&st->amt_max, amax);
-            atomicMin(&st->ent_min, emin); atomicMax(&st->ent_max, emax);
-            atomicMin(&st->w_min, wmin); atomicMax(&st->w_max, wmax);
-            atomicMin(&st->d_min, dmin); atomicMax(&st->d_max, dmax);
-            atomicMin(&st->o_min, omin); atomicMax(&st->o_max, omax);
+    }
+    __device__ Q18Stats get() const {
+        Q18Stats s;
+        s.amt_min = amin; s.amt_max = amax; s.ent_min = emin; s.ent_max = emax;
+        s.w_min = wmin; s.w_max = wmax; s.d_min = dmin; s.d_max = dmax; s.o_min = omin; s.o_max = omax;
+        s.pad0 = s.pad1 = 0;
+        return s;
+    }
+    // Block reduction into part[blockIdx.x]; the last block to finish folds every block's
+    // partial into *out (no same-address atomics: thousands of warps would serialise on them).
+    __device__ void flush(Q18Stats *part, unsigned int *ticket, Q18Stats *out) {
+        __shared__ Q18Stats ws[32];
+        __shared__ bool last;
+        const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5, nw = (blockDim.x + 31) >> 5;
+        warp_reduce();
+        if (lane == 0) ws[warp] = get();
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            StatAcc b;
+            for (int k = 0; k < nw; ++k) b.merge(ws[k]);
+            part[blockIdx.x] = b.get();
+            __threadfence();
+            last = atomicAdd(ticket, 1u) == gridDim.x - 1;
+        }
+        __syncthreads();
+        if (!last) return;
+        __threadfence();
+        StatAcc f;
+        for (unsigned k = threadIdx.x; k < gridDim.x; k += blockDim.x) {
+            Q18Stats x;
+            const long long *src = reinterpret_cast<const long long *>(part + k);
+            long long *dst = reinterpret_cast<long long *>(&x);
+            for (int q = 0; q < (int)(sizeof(Q18Stats) / 8); ++q) dst[q] = __ldcg(src + q);
+            f.merge(x);
+        }
+        f.warp_reduce();
+        __syncthreads();
+        if (lane == 0) ws[warp] = f.get();
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            StatAcc b;
+            for (int k = 0; k < nw; ++k) b.merge(ws[k]);
+            *out = b.get();
+            *ticket = 0;  // self-reset for the next launch
         }
     }
 };
@@ -232,10 +306,10 @@ struct StatAcc {
 // Each block iteration covers kHavingRows consecutive orders rows (kHavingUnroll per thread);
 // passing rows get output slots from ONE atomicAdd per block iteration (block-wide exclusive
 // scan of the per-thread counts), so the output counter sees ~n/1024 atomics, not n/32.
-constexpr int kHavingUnroll = 4;
+constexpr int kHavingUnroll = 2;
 constexpr int kHavingRows = kHavingThreads * kHavingUnroll;
 
-__global__ void __launch_bounds__(kHavingThreads)
+__global__ void __launch_bounds__(kHavingThreads, 4)
 q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
                   const int32_t *__restrict__ o_id, const int32_t *__restrict__ o_c,
                   const int32_t *__restrict__ o_cnt, const int64_t *__restrict__ o_ent, uint64_t n,
@@ -249,22 +323,27 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
         unsigned int crow[kHavingUnroll];
         long long sum[kHavingUnroll];
         int w[kHavingUnroll], d[kHavingUnroll], c[kHavingUnroll];
+        bool pass1[kHavingUnroll];
         unsigned int mine = 0;
+        // stage 1: independent coalesced loads for all rows (maximise loads in flight)
 #pragma unroll
         for (int u = 0; u < kHavingUnroll; ++u) {
             const uint64_t r = base + u * kHavingThreads + threadIdx.x;
-            crow[u] = kNoRow;
+            pass1[u] = false;
             sum[u] = 0;
             w[u] = d[u] = c[u] = 0;
             if (r < n) {
                 const ulonglong2 a = __ldcs(reinterpret_cast<const ulonglong2 *>(s.acc + r));
                 sum[u] = (long long)a.x;
                 // inner join: a group exists only with >= 1 order_line row; HAVING SUM > having
-                if ((unsigned int)a.y > 0 && sum[u] > having) {
-                    w[u] = o_w[r]; d[u] = o_d[r]; c[u] = o_c[r];
-                    crow[u] = jx_lookup(s.jc, w[u], d[u], c[u]);  // customer ⋈ orders
-                }
+                pass1[u] = (unsigned int)a.y > 0 && sum[u] > having;
+                w[u] = __ldcs(o_w + r); d[u] = __ldcs(o_d + r); c[u] = __ldcs(o_c + r);
             }
+        }
+        // stage 2: customer ⋈ orders lookups, independent across rows
+#pragma unroll
+        for (int u = 0; u < kHavingUnroll; ++u) {
+            crow[u] = pass1[u] ? jx_lookup(s.jc, w[u], d[u], c[u]) : kNoRow;
             mine += crow[u] != kNoRow;
         }
         // block-wide exclusive scan of `mine`, one atomic for the block's output range
@@ -285,35 +364,40 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
         if (threadIdx.x == 0) s_base = total ? atomicAdd(s.nout, (unsigned long long)total) : 0ull;
         __syncthreads();
         uint64_t p = s_base + before + x - mine;
+        Q18Row row[kHavingUnroll];
+#pragma unroll
+        for (int u = 0; u < kHavingUnroll; ++u) {  // stage 3: gathers for passing rows
+            if (crow[u] == kNoRow) continue;
+            const uint64_t r = base + u * kHavingThreads + threadIdx.x;
+            row[u].o_entry_d = __ldcs(o_ent + r);
+            row[u].c_last = __ldg(c_last + crow[u]);
+            row[u].c_id = c[u];
+            row[u].o_id = __ldcs(o_id + r);
+            row[u].o_ol_cnt = __ldcs(o_cnt + r);
+            row[u].o_w_id = w[u];
+            row[u].o_d_id = d[u];
+        }
 #pragma unroll
         for (int u = 0; u < kHavingUnroll; ++u) {
             if (crow[u] == kNoRow) continue;
-            const uint64_t r = base + u * kHavingThreads + threadIdx.x;
-            Q18Row row;
-            row.amount_sum = sum[u];
-            row.o_entry_d = o_ent[r];
-            row.c_last = c_last[crow[u]];
-            row.c_id = c[u];
-            row.o_id = o_id[r];
-            row.o_ol_cnt = o_cnt[r];
-            row.o_w_id = w[u];
-            row.o_d_id = d[u];
-            s.rows[p++] = row;
-            stat.add(sum[u], row.o_entry_d, w[u], d[u], row.o_id);
+            s.amt[p] = sum[u];
+            s.rows[p++] = row[u];
+            stat.add(sum[u], row[u].o_entry_d, w[u], d[u], row[u].o_id);
         }
         __syncthreads();  // wsum / s_base reuse
     }
-    stat.flush(s.stats);
+    stat.flush(s.stat_part, s.ticket, s.stats);
 }
 
-__global__ void q18_stats_kernel(const Q18Row *__restrict__ rows, uint64_t n, Q18Stats *st) {
+__global__ void q18_stats_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
+                                 uint64_t n, Q18Stats *st, Q18Stats *part, unsigned int *ticket) {
     StatAcc stat;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
         const Q18Row r = rows[i];
-        stat.add(r.amount_sum, r.o_entry_d, r.o_w_id, r.o_d_id, r.o_id);
+        stat.add(amt[i], r.o_entry_d, r.o_w_id, r.o_d_id, r.o_id);
     }
-    stat.flush(st);
+    stat.flush(part, ticket, st);
 }
 
 }  // namespace
@@ -335,8 +419,8 @@ void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_i
 void launch_q18_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
                       const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
                       cudaStream_t st) {
-    q18_probe_kernel<<<grid_for((n_ol + kProbeUnroll - 1) / kProbeUnroll, kProbeThreads, num_sms, 8),
-                       kProbeThreads, 0, st>>>(ol_w, ol_d, ol_o, ol_amt, n_ol, s);
+    q18_probe_kernel<<<grid_for((n_ol + 3) / 4, kProbeThreads, num_sms, 8), kProbeThreads, 0, st>>>(
+        ol_w, ol_d, ol_o, ol_amt, n_ol, s);
     count_launches(1);
 }
 
@@ -350,9 +434,10 @@ void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_
     count_launches(1);
 }
 
-void launch_q18_stats(const Q18Row *rows, uint64_t n, Q18Stats *stats, int num_sms,
-                      cudaStream_t st) {
-    q18_stats_kernel<<<grid_for(n, 256, num_sms, 4), 256, 0, st>>>(rows, n, stats);
+void launch_q18_stats(const Q18Row *rows, const long long *amt, uint64_t n, const Q18Scratch &s,
+                      int num_sms, cudaStream_t st) {
+    q18_stats_kernel<<<grid_for(n, 256, num_sms, 4), 256, 0, st>>>(rows, amt, n, s.stats, s.stat_part,
+                                                                  s.ticket);
     count_launches(1);
 }
 

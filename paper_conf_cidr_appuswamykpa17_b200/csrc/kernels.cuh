@@ -71,10 +71,11 @@ struct Q18Stats {            // min/max of the sort fields over result rows (ato
     long long amt_min, amt_max, ent_min, ent_max;
     int w_min, w_max, d_min, d_max, o_min, o_max, pad0, pad1;
 };
-struct Q18Row {              // one result row before ORDER BY (AoS: one 40-byte gather later)
-    long long amount_sum, o_entry_d;
-    int c_last, c_id, o_id, o_ol_cnt, o_w_id, o_d_id;
+struct __align__(16) Q18Row {  // one result row before ORDER BY: 32 B = one L2 sector per gather
+    long long o_entry_d;       // (amount_sum lives in a parallel array: after the sort it is
+    int c_last, c_id, o_id, o_ol_cnt, o_w_id, o_d_id;  //  recovered from the sorted key)
 };
+static_assert(sizeof(Q18Row) == 32, "Q18Row must be one sector");
 struct Q18Cols {             // SoA result columns
     int32_t *c_last, *c_id, *o_id, *o_ol_cnt, *o_w_id, *o_d_id;
     int64_t *o_entry_d, *amount_sum;
@@ -84,8 +85,11 @@ struct Q18Scratch {
     Q18Acc *acc;             // [n_orders]
     unsigned int *err;       // [1]
     unsigned long long *nout;// [1]
-    Q18Stats *stats;         // [1]
+    Q18Stats *stats;         // [1] final
+    Q18Stats *stat_part;     // [grid] per-block partials
+    unsigned int *ticket;    // [1] last-block counter, zero-initialised once, self-resetting
     Q18Row *rows;            // [n_orders] unsorted result rows
+    long long *amt;          // [n_orders] their amount_sum
 };
 void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st);
 void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
@@ -98,8 +102,8 @@ void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_
                        const int32_t *o_c, const int32_t *o_cnt, const int64_t *o_ent,
                        uint64_t n_o, const int32_t *c_last, int64_t having,
                        const Q18Scratch &s, int num_sms, cudaStream_t st);
-void launch_q18_stats(const Q18Row *rows, uint64_t n, Q18Stats *stats, int num_sms,
-                      cudaStream_t st);  // recompute stats over gathered rows (multi-GPU)
+void launch_q18_stats(const Q18Row *rows, const long long *amt, uint64_t n, const Q18Scratch &s,
+                      int num_sms, cudaStream_t st);  // recompute stats over gathered rows (multi-GPU)
 
 // ------------------------------------------------------------------ sort ---
 // Stable LSD radix sort of (u64 key, u32 value) pairs, 8-bit digits, `bits` low key bits.
@@ -119,14 +123,15 @@ int radix_sort_pairs(uint64_t n, int bits, const SortPairs &s, int num_sms, cuda
 
 // Bucket sort of (u64 key, u32 value) pairs whose keys use the low `bits` bits: partition by the
 // top `bucket_bits` key bits (histogram -> scan -> scatter), then sort every bucket in shared
-// memory (bitonic). A bucket larger than kBucketCap raises *flag (caller falls back to LSD).
-constexpr int kBucketCap = 8192;
+// memory (two-level: sub-buckets + rank). A bucket larger than 4096 rows raises *flag (the caller
+// falls back to the exact LSD sort).
+constexpr int kBucketMaxBits = 15;
 struct BucketSort {
     unsigned long long *k[2];
     unsigned int *v[2];
-    unsigned int *count;   // [2^bucket_bits + 1]
-    unsigned int *cursor;  // [2^bucket_bits]
-    unsigned int *offset;  // [2^bucket_bits + 1]
+    unsigned int *count;   // [2^kBucketMaxBits + 1]
+    unsigned int *cursor;  // [2^kBucketMaxBits]
+    unsigned int *offset;  // [2^kBucketMaxBits + 1]
 };
 // Sorted pairs end in k[1]/v[1] (input in k[0]/v[0]).
 void bucket_sort_pairs(uint64_t n, int bits, int bucket_bits, const BucketSort &s, unsigned int *flag,
@@ -140,17 +145,21 @@ struct Q18SortSpec {         // host-computed from Q18Stats
     int bits_a, bits_e, bits_r;  // field widths: amount (desc), entry, row rank
     int prefix_bits;         // width of the sorted 64-bit prefix of the composite key
 };
-void launch_q18_sort_keys(const Q18Row *rows, uint64_t n, const Q18SortSpec &spec,
-                          const SortPairs &s, int num_sms, cudaStream_t st);
+void launch_q18_sort_keys(const Q18Row *rows, const long long *amt, uint64_t n,
+                          const Q18SortSpec &spec, const SortPairs &s, int num_sms, cudaStream_t st);
 // Within runs of equal prefix, order by the full tuple; runs longer than 32 raise *flag.
-void launch_q18_tiefix(const Q18Row *rows, const unsigned long long *keys, unsigned int *vals,
-                       uint64_t n, unsigned int *flag, int num_sms, cudaStream_t st);
+void launch_q18_tiefix(const Q18Row *rows, const long long *amt, const unsigned long long *keys,
+                       unsigned int *vals, uint64_t n, unsigned int *flag, int num_sms,
+                       cudaStream_t st);
 // Exact fallback: three stable passes over the full fields (row rank, entry, amount).
-void launch_q18_field_keys(const Q18Row *rows, const unsigned int *vals, uint64_t n, int field,
-                           const Q18SortSpec &spec, unsigned long long *keys, int num_sms,
-                           cudaStream_t st);
+void launch_q18_field_keys(const Q18Row *rows, const long long *amt, const unsigned int *vals,
+                           uint64_t n, int field, const Q18SortSpec &spec, unsigned long long *keys,
+                           int num_sms, cudaStream_t st);
 void launch_iota(unsigned int *v, uint64_t n, int num_sms, cudaStream_t st);
-void launch_q18_permute(const Q18Row *rows, const unsigned int *perm, uint64_t n,
+// Gather rows in `perm` order into SoA columns. amount_sum: decoded from the sorted prefix keys
+// when `keys` is given (field a is always whole at the top of the prefix), else read from amt.
+void launch_q18_permute(const Q18Row *rows, const long long *amt, const unsigned int *perm,
+                        const unsigned long long *keys, const Q18SortSpec &spec, uint64_t n,
                         const Q18Cols &dst, int num_sms, cudaStream_t st);
 
 // ------------------------------------------------------------ store (a1) --

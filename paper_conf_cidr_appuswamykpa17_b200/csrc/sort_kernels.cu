@@ -154,8 +154,8 @@ scatter_kernel(const unsigned long long *__restrict__ kin, const unsigned int *_
 }
 
 // ------------------------------------------------------------ Q18 keys --
-__device__ __forceinline__ unsigned long long field_a(const Q18Row &r, const Q18SortSpec &sp) {
-    return (unsigned long long)sp.amt_max - (unsigned long long)r.amount_sum;  // DESC
+__device__ __forceinline__ unsigned long long field_a(long long amount, const Q18SortSpec &sp) {
+    return (unsigned long long)sp.amt_max - (unsigned long long)amount;  // DESC
 }
 __device__ __forceinline__ unsigned long long field_e(const Q18Row &r, const Q18SortSpec &sp) {
     return (unsigned long long)r.o_entry_d - (unsigned long long)sp.ent_min;
@@ -168,8 +168,9 @@ __device__ __forceinline__ unsigned long long field_r(const Q18Row &r, const Q18
 }
 
 // top `prefix_bits` bits of the concatenation (a | e | r) with widths (bits_a, bits_e, bits_r)
-__device__ __forceinline__ unsigned long long prefix_key(const Q18Row &r, const Q18SortSpec &sp) {
-    const unsigned long long f[3] = {field_a(r, sp), field_e(r, sp), field_r(r, sp)};
+__device__ __forceinline__ unsigned long long prefix_key(const Q18Row &r, long long amount,
+                                                         const Q18SortSpec &sp) {
+    const unsigned long long f[3] = {field_a(amount, sp), field_e(r, sp), field_r(r, sp)};
     const int b[3] = {sp.bits_a, sp.bits_e, sp.bits_r};
     unsigned long long p = 0;
     int room = sp.prefix_bits;
@@ -184,18 +185,19 @@ __device__ __forceinline__ unsigned long long prefix_key(const Q18Row &r, const 
     return p;
 }
 
-__global__ void sort_keys_kernel(const Q18Row *__restrict__ rows, uint64_t n, Q18SortSpec sp,
-                                 unsigned long long *__restrict__ k, unsigned int *__restrict__ v) {
+__global__ void sort_keys_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
+                                 uint64_t n, Q18SortSpec sp, unsigned long long *__restrict__ k,
+                                 unsigned int *__restrict__ v) {
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
-        k[i] = prefix_key(rows[i], sp);
+        k[i] = prefix_key(rows[i], amt[i], sp);
         v[i] = (unsigned int)i;
     }
 }
 
 // full ORDER BY comparison: amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id
-__device__ __forceinline__ bool row_less(const Q18Row &x, const Q18Row &y) {
-    if (x.amount_sum != y.amount_sum) return x.amount_sum > y.amount_sum;
+__device__ __forceinline__ bool row_less(const Q18Row &x, long long ax, const Q18Row &y, long long ay) {
+    if (ax != ay) return ax > ay;
     if (x.o_entry_d != y.o_entry_d) return x.o_entry_d < y.o_entry_d;
     if (x.o_w_id != y.o_w_id) return x.o_w_id < y.o_w_id;
     if (x.o_d_id != y.o_d_id) return x.o_d_id < y.o_d_id;
@@ -204,8 +206,9 @@ __device__ __forceinline__ bool row_less(const Q18Row &x, const Q18Row &y) {
 
 constexpr int kMaxRun = 32;
 
-__global__ void tiefix_kernel(const Q18Row *__restrict__ rows, const unsigned long long *__restrict__ k,
-                              unsigned int *__restrict__ v, uint64_t n, unsigned int *flag) {
+__global__ void tiefix_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
+                              const unsigned long long *__restrict__ k, unsigned int *__restrict__ v,
+                              uint64_t n, unsigned int *flag) {
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
         const unsigned long long ki = k[i];
@@ -220,21 +223,23 @@ __global__ void tiefix_kernel(const Q18Row *__restrict__ rows, const unsigned lo
         for (int t = 1; t < len; ++t) {  // insertion sort by the full tuple
             const unsigned int x = idx[t];
             const Q18Row rx = rows[x];
+            const long long ax = amt[x];
             int u = t - 1;
-            while (u >= 0 && row_less(rx, rows[idx[u]])) { idx[u + 1] = idx[u]; --u; }
+            while (u >= 0 && row_less(rx, ax, rows[idx[u]], amt[idx[u]])) { idx[u + 1] = idx[u]; --u; }
             idx[u + 1] = x;
         }
         for (int t = 0; t < len; ++t) v[i + t] = idx[t];
     }
 }
 
-__global__ void field_keys_kernel(const Q18Row *__restrict__ rows, const unsigned int *__restrict__ vals,
-                                  uint64_t n, int field, Q18SortSpec sp,
-                                  unsigned long long *__restrict__ k) {
+__global__ void field_keys_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
+                                  const unsigned int *__restrict__ vals, uint64_t n, int field,
+                                  Q18SortSpec sp, unsigned long long *__restrict__ k) {
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
-        const Q18Row r = rows[vals[i]];
-        k[i] = field == 0 ? field_r(r, sp) : field == 1 ? field_e(r, sp) : field_a(r, sp);
+        const unsigned int x = vals[i];
+        const Q18Row r = rows[x];
+        k[i] = field == 0 ? field_r(r, sp) : field == 1 ? field_e(r, sp) : field_a(amt[x], sp);
     }
 }
 
@@ -244,18 +249,30 @@ __global__ void iota_kernel(unsigned int *v, uint64_t n) {
         v[i] = (unsigned int)i;
 }
 
-// Gather one 40-byte row per output position, write the eight SoA columns coalesced.
-__global__ void permute_kernel(const Q18Row *__restrict__ rows, const unsigned int *__restrict__ perm,
+// Gather one 32-byte row (one sector) per output position, write the SoA columns coalesced;
+// amount_sum comes from the sorted prefix key (contiguous) instead of a second random gather.
+__global__ void permute_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
+                               const unsigned int *__restrict__ perm,
+                               const unsigned long long *__restrict__ keys, Q18SortSpec sp,
                                uint64_t n, Q18Cols dst) {
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    const int ashift = sp.prefix_bits - sp.bits_a;
     for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < n; j += stride) {
-        const Q18Row r = rows[perm ? perm[j] : j];
+        const unsigned int i = perm ? perm[j] : (unsigned int)j;
+        const Q18Row r = rows[i];
+        long long amount;
+        if (keys) {
+            const unsigned long long a = sp.bits_a ? (__ldcs(keys + j) >> ashift) : 0ull;
+            amount = (long long)((unsigned long long)sp.amt_max - a);
+        } else {
+            amount = amt[i];
+        }
         dst.c_last[j] = r.c_last;
         dst.c_id[j] = r.c_id;
         dst.o_id[j] = r.o_id;
         dst.o_entry_d[j] = r.o_entry_d;
         dst.o_ol_cnt[j] = r.o_ol_cnt;
-        dst.amount_sum[j] = r.amount_sum;
+        dst.amount_sum[j] = amount;
         dst.o_w_id[j] = r.o_w_id;
         dst.o_d_id[j] = r.o_d_id;
     }
@@ -287,22 +304,23 @@ int radix_sort_pairs(uint64_t n, int bits, const SortPairs &s, int num_sms, cuda
     return cur;
 }
 
-void launch_q18_sort_keys(const Q18Row *rows, uint64_t n, const Q18SortSpec &spec,
-                          const SortPairs &s, int num_sms, cudaStream_t st) {
-    sort_keys_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, n, spec, s.k[0], s.v[0]);
+void launch_q18_sort_keys(const Q18Row *rows, const long long *amt, uint64_t n,
+                          const Q18SortSpec &spec, const SortPairs &s, int num_sms, cudaStream_t st) {
+    sort_keys_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, amt, n, spec, s.k[0], s.v[0]);
     count_launches(1);
 }
 
-void launch_q18_tiefix(const Q18Row *rows, const unsigned long long *keys, unsigned int *vals,
-                       uint64_t n, unsigned int *flag, int num_sms, cudaStream_t st) {
-    tiefix_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, keys, vals, n, flag);
+void launch_q18_tiefix(const Q18Row *rows, const long long *amt, const unsigned long long *keys,
+                       unsigned int *vals, uint64_t n, unsigned int *flag, int num_sms,
+                       cudaStream_t st) {
+    tiefix_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, amt, keys, vals, n, flag);
     count_launches(1);
 }
 
-void launch_q18_field_keys(const Q18Row *rows, const unsigned int *vals, uint64_t n, int field,
-                           const Q18SortSpec &spec, unsigned long long *keys, int num_sms,
-                           cudaStream_t st) {
-    field_keys_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, vals, n, field, spec, keys);
+void launch_q18_field_keys(const Q18Row *rows, const long long *amt, const unsigned int *vals,
+                           uint64_t n, int field, const Q18SortSpec &spec, unsigned long long *keys,
+                           int num_sms, cudaStream_t st) {
+    field_keys_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, amt, vals, n, field, spec, keys);
     count_launches(1);
 }
 
@@ -311,9 +329,10 @@ void launch_iota(unsigned int *v, uint64_t n, int num_sms, cudaStream_t st) {
     count_launches(1);
 }
 
-void launch_q18_permute(const Q18Row *rows, const unsigned int *perm, uint64_t n,
+void launch_q18_permute(const Q18Row *rows, const long long *amt, const unsigned int *perm,
+                        const unsigned long long *keys, const Q18SortSpec &spec, uint64_t n,
                         const Q18Cols &dst, int num_sms, cudaStream_t st) {
-    permute_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, perm, n, dst);
+    permute_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, amt, perm, keys, spec, n, dst);
     count_launches(1);
 }
 
@@ -321,15 +340,19 @@ void launch_q18_permute(const Q18Row *rows, const unsigned int *perm, uint64_t n
 
 // ============================================================ bucket sort ===
 // Main ORDER BY path: the result (a few million 12-byte pairs) fits in L2, so
-// one partition pass by the top key bits plus a shared-memory sort per bucket replaces the
-// 6 LSD passes. Buckets are not stable internally; equal full prefixes are ordered afterwards by
-// the tie-fix kernel (which sorts runs of equal prefix by the full tuple) — so the result is the
-// same total order as the LSD path.
+// one partition pass by the top key bits plus a shared-memory sort per bucket replaces LSD
+// passes. Inside a bucket: a second partition by the next bits into sub-buckets of ~8 rows, then
+// every row's final position is its rank inside its sub-bucket (count of smaller keys, ties by
+// position) — no barriers inside the ranking. Equal 64-bit prefixes are ordered afterwards by
+// the tie-fix kernel (full tuple), so the result is the same total order as the LSD path.
 namespace h2tap {
 namespace {
 
 constexpr int kBkThreads = 256;
-constexpr int kBkSmemBins = 8192;  // max buckets counted in shared memory per block
+constexpr int kBkItems = 16;                       // rows per thread in hist/scatter
+constexpr int kLsCapSmall = 2048;                  // rows per bucket: fast kernel (3 blocks/SM)
+constexpr int kLsCapLarge = 8192;                  // rows per bucket: large-bucket kernel
+constexpr int kLsSubMax = 1024;                    // max sub-buckets per bucket
 
 __global__ void __launch_bounds__(kBkThreads)
 bucket_hist_kernel(const unsigned long long *__restrict__ key, uint64_t n, int shift, int nb,
@@ -337,9 +360,18 @@ bucket_hist_kernel(const unsigned long long *__restrict__ key, uint64_t n, int s
     extern __shared__ unsigned int h[];
     for (int i = threadIdx.x; i < nb; i += kBkThreads) h[i] = 0;
     __syncthreads();
-    const uint64_t stride = (uint64_t)gridDim.x * kBkThreads;
-    for (uint64_t i = (uint64_t)blockIdx.x * kBkThreads + threadIdx.x; i < n; i += stride)
-        atomicAdd(&h[(unsigned int)(__ldcg(key + i) >> shift)], 1u);
+    for (uint64_t base = (uint64_t)blockIdx.x * kBkThreads * kBkItems; base < n;
+         base += (uint64_t)gridDim.x * kBkThreads * kBkItems) {
+        unsigned int b[kBkItems];
+#pragma unroll
+        for (int i = 0; i < kBkItems; ++i) {
+            const uint64_t j = base + (uint64_t)i * kBkThreads + threadIdx.x;
+            b[i] = j < n ? (unsigned int)(__ldcg(key + j) >> shift) : 0xffffffffu;
+        }
+#pragma unroll
+        for (int i = 0; i < kBkItems; ++i)
+            if (b[i] != 0xffffffffu) atomicAdd(&h[b[i]], 1u);
+    }
     __syncthreads();
     for (int i = threadIdx.x; i < nb; i += kBkThreads)
         if (h[i]) atomicAdd(count + i, h[i]);
@@ -392,68 +424,129 @@ __global__ void __launch_bounds__(1024) bucket_scan_kernel(unsigned int *__restr
     }
 }
 
-// scatter into buckets: per-block shared histogram reserves one global range per bucket
+// scatter into buckets: a block's shared histogram reserves one global range per bucket
 __global__ void __launch_bounds__(kBkThreads)
 bucket_scatter_kernel(const unsigned long long *__restrict__ kin, const unsigned int *__restrict__ vin,
                       unsigned long long *__restrict__ kout, unsigned int *__restrict__ vout, uint64_t n,
-                      int shift, int nb, unsigned int *__restrict__ cursor, uint64_t per_block) {
+                      int shift, int nb, unsigned int *__restrict__ cursor) {
     extern __shared__ unsigned int h[];  // [nb] local counts -> local cursors
     for (int i = threadIdx.x; i < nb; i += kBkThreads) h[i] = 0;
+    const uint64_t base = (uint64_t)blockIdx.x * kBkThreads * kBkItems;
+    unsigned long long k[kBkItems];
+    unsigned int b[kBkItems];
+#pragma unroll
+    for (int i = 0; i < kBkItems; ++i) {
+        const uint64_t j = base + (uint64_t)i * kBkThreads + threadIdx.x;
+        k[i] = j < n ? __ldcs(kin + j) : 0ull;
+        b[i] = j < n ? (unsigned int)(k[i] >> shift) : 0xffffffffu;
+    }
     __syncthreads();
-    const uint64_t lo = (uint64_t)blockIdx.x * per_block;
-    const uint64_t hi = lo + per_block < n ? lo + per_block : n;
-    for (uint64_t i = lo + threadIdx.x; i < hi; i += kBkThreads)
-        atomicAdd(&h[(unsigned int)(__ldcg(kin + i) >> shift)], 1u);
+#pragma unroll
+    for (int i = 0; i < kBkItems; ++i)
+        if (b[i] != 0xffffffffu) atomicAdd(&h[b[i]], 1u);
     __syncthreads();
-    for (int i = threadIdx.x; i < nb; i += kBkThreads)
+#pragma unroll 8
+    for (int i = threadIdx.x; i < nb; i += kBkThreads)  // independent atomics: keep 8 in flight
         if (h[i]) h[i] = atomicAdd(cursor + i, h[i]);  // base of this block's range in bucket i
     __syncthreads();
-    for (uint64_t i = lo + threadIdx.x; i < hi; i += kBkThreads) {
-        const unsigned long long k = __ldcg(kin + i);
-        const unsigned int p = atomicAdd(&h[(unsigned int)(k >> shift)], 1u);
-        kout[p] = k;
-        vout[p] = __ldcg(vin + i);
+#pragma unroll
+    for (int i = 0; i < kBkItems; ++i) {
+        if (b[i] == 0xffffffffu) continue;
+        const uint64_t j = base + (uint64_t)i * kBkThreads + threadIdx.x;
+        const unsigned int p = atomicAdd(&h[b[i]], 1u);
+        kout[p] = k[i];
+        vout[p] = __ldcs(vin + j);
     }
 }
 
-// one block per bucket: load into shared memory, bitonic sort by key, write back
+template <int kLsCap> struct LsSmem {
+    unsigned long long k1[kLsCap], k2[kLsCap];
+    unsigned int v1[kLsCap], v2[kLsCap];
+    unsigned int sub[kLsSubMax + 1];   // sub-bucket counts -> offsets
+    unsigned int cur[kLsSubMax];       // sub-bucket cursors
+    unsigned int wsum[kBkThreads / 32];
+};
+
+// One block per bucket: load it into shared memory, partition by the next `sb` key bits into
+// sub-buckets, write every row at offset + its rank within its sub-bucket. The kernel handles
+// buckets of (kMin, kLsCap] rows; the large instance flags buckets above its capacity.
+template <int kLsCap, int kMin>
 __global__ void __launch_bounds__(kBkThreads)
 bucket_local_sort_kernel(unsigned long long *__restrict__ k, unsigned int *__restrict__ v,
-                         const unsigned int *__restrict__ offset, int nb, unsigned int *flag) {
-    extern __shared__ unsigned long long sk[];  // [kBucketCap] keys, then [kBucketCap] values
-    unsigned int *sv = reinterpret_cast<unsigned int *>(sk + kBucketCap);
+                         const unsigned int *__restrict__ offset, int nb, int shift,
+                         unsigned int *flag) {
+    extern __shared__ __align__(16) unsigned char smem_raw[];
+    LsSmem<kLsCap> &S = *reinterpret_cast<LsSmem<kLsCap> *>(smem_raw);
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     for (int b = blockIdx.x; b < nb; b += gridDim.x) {
-        const unsigned int lo = offset[b], cnt = offset[b + 1] - lo;
-        if (cnt <= 1) continue;
-        if (cnt > (unsigned)kBucketCap) {
-            if (threadIdx.x == 0) atomicOr(flag, 2u);
+        const unsigned int lo = offset[b], m = offset[b + 1] - lo;
+        if (m <= (unsigned)(kMin > 1 ? kMin : 1)) continue;
+        if (m > (unsigned)kLsCap) {
+            if (threadIdx.x == 0 && kMin > 0) atomicOr(flag, 2u);  // only the large instance flags
             continue;
         }
-        unsigned int m = 2;
-        while (m < cnt) m <<= 1;
+        // sub-bucket bits: ~8 rows per sub-bucket, at most kLsSubMax sub-buckets
+        int sb = 0;
+        while (sb < 10 && (m >> (sb + 3)) > 0) ++sb;
+        if (sb > shift) sb = shift;
+        const int ssh = shift - sb;
+        const unsigned int ns = 1u << sb, smask = ns - 1u;
+        for (unsigned int i = threadIdx.x; i < ns; i += kBkThreads) S.sub[i] = 0;
+        __syncthreads();
         for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
-            sk[i] = i < cnt ? k[lo + i] : ~0ull;
-            sv[i] = i < cnt ? v[lo + i] : 0u;
+            const unsigned long long kk = k[lo + i];
+            S.k1[i] = kk;
+            S.v1[i] = v[lo + i];
+            atomicAdd(&S.sub[(unsigned int)(kk >> ssh) & smask], 1u);
         }
         __syncthreads();
-        for (unsigned int size = 2; size <= m; size <<= 1) {
-            for (unsigned int stride = size >> 1; stride > 0; stride >>= 1) {
-                for (unsigned int t = threadIdx.x; t < m / 2; t += kBkThreads) {
-                    const unsigned int i = 2 * t - (t & (stride - 1));
-                    const unsigned int j = i + stride;
-                    const bool up = (i & size) == 0;
-                    const unsigned long long a = sk[i], c = sk[j];
-                    if ((a > c) == up) {
-                        sk[i] = c; sk[j] = a;
-                        const unsigned int tv = sv[i]; sv[i] = sv[j]; sv[j] = tv;
-                    }
-                }
-                __syncthreads();
+        // exclusive scan of ns (<= 1024) sub-bucket counts: 4 per thread
+        {
+            unsigned int c[4], t = 0;
+#pragma unroll
+            for (int q = 0; q < 4; ++q) {
+                const unsigned int i = threadIdx.x * 4 + q;
+                c[q] = i < ns ? S.sub[i] : 0u;
+                t += c[q];
             }
+            unsigned int x = t;
+#pragma unroll
+            for (int o = 1; o < 32; o <<= 1) {
+                const unsigned int y = __shfl_up_sync(kFull, x, o);
+                if (lane >= o) x += y;
+            }
+            if (lane == 31) S.wsum[warp] = x;
+            __syncthreads();
+            unsigned int before = 0;
+            for (int w = 0; w < warp; ++w) before += S.wsum[w];
+            unsigned int run = before + x - t;
+#pragma unroll
+            for (int q = 0; q < 4; ++q) {
+                const unsigned int i = threadIdx.x * 4 + q;
+                if (i < ns) { S.sub[i] = run; S.cur[i] = run; }
+                run += c[q];
+            }
+            if (threadIdx.x == kBkThreads - 1) S.sub[ns] = run;
         }
-        for (unsigned int i = threadIdx.x; i < cnt; i += kBkThreads) {
-            k[lo + i] = sk[i];
-            v[lo + i] = sv[i];
+        __syncthreads();
+        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
+            const unsigned long long kk = S.k1[i];
+            const unsigned int p = atomicAdd(&S.cur[(unsigned int)(kk >> ssh) & smask], 1u);
+            S.k2[p] = kk;
+            S.v2[p] = S.v1[i];
+        }
+        __syncthreads();
+        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
+            const unsigned long long kk = S.k2[i];
+            const unsigned int sbk = (unsigned int)(kk >> ssh) & smask;
+            const unsigned int s0 = S.sub[sbk], s1 = S.sub[sbk + 1];
+            unsigned int rank = s0;
+            for (unsigned int j = s0; j < s1; ++j) {
+                const unsigned long long kj = S.k2[j];
+                rank += (kj < kk) | ((kj == kk) & (j < i));
+            }
+            k[lo + rank] = kk;
+            v[lo + rank] = S.v2[i];
         }
         __syncthreads();
     }
@@ -464,30 +557,42 @@ bucket_local_sort_kernel(unsigned long long *__restrict__ k, unsigned int *__res
 void bucket_sort_pairs(uint64_t n, int bits, int bucket_bits, const BucketSort &s, unsigned int *flag,
                        int num_sms, cudaStream_t st) {
     if (bucket_bits > bits) bucket_bits = bits;
-    if (bucket_bits > 13) bucket_bits = 13;  // shared histogram of <= 8192 bins
+    if (bucket_bits > kBucketMaxBits) bucket_bits = kBucketMaxBits;
     const int nb = 1 << bucket_bits;
     const int shift = bits - bucket_bits;
     static bool init = false;
     if (!init) {
-        cudaFuncSetAttribute(bucket_local_sort_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                             kBucketCap * 12);
+        cudaFuncSetAttribute(bucket_local_sort_kernel<kLsCapSmall, 0>,
+                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapSmall>));
+        cudaFuncSetAttribute(bucket_local_sort_kernel<kLsCapLarge, kLsCapSmall>,
+                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapLarge>));
+        cudaFuncSetAttribute(bucket_hist_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             4 << kBucketMaxBits);
+        cudaFuncSetAttribute(bucket_scatter_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             4 << kBucketMaxBits);
         init = true;
     }
     cudaMemsetAsync(s.count, 0, sizeof(unsigned int) * (nb + 1), st);
-    uint64_t hb = (n + kBkThreads * 16 - 1) / (kBkThreads * 16);
-    if (hb > (uint64_t)num_sms * 4) hb = (uint64_t)num_sms * 4;
+    const uint64_t per = (uint64_t)kBkThreads * kBkItems;
+    uint64_t hb = (n + per - 1) / per;
+    if (hb > (uint64_t)num_sms * 2) hb = (uint64_t)num_sms * 2;
     if (!hb) hb = 1;
     bucket_hist_kernel<<<(unsigned)hb, kBkThreads, nb * 4, st>>>(s.k[0], n, shift, nb, s.count);
     count_launches(1);
     bucket_scan_kernel<<<1, 1024, 0, st>>>(s.count, nb, s.offset, s.cursor);
     count_launches(1);
-    const uint64_t per_block = 16384;
-    const uint64_t sb = (n + per_block - 1) / per_block;
+    const uint64_t sb = (n + per - 1) / per;
     bucket_scatter_kernel<<<(unsigned)(sb ? sb : 1), kBkThreads, nb * 4, st>>>(
-        s.k[0], s.v[0], s.k[1], s.v[1], n, shift, nb, s.cursor, per_block);
+        s.k[0], s.v[0], s.k[1], s.v[1], n, shift, nb, s.cursor);
     count_launches(1);
-    unsigned lb = (unsigned)nb < (unsigned)num_sms * 16 ? (unsigned)nb : (unsigned)num_sms * 16;
-    bucket_local_sort_kernel<<<lb, kBkThreads, kBucketCap * 12, st>>>(s.k[1], s.v[1], s.offset, nb, flag);
+    unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
+    bucket_local_sort_kernel<kLsCapSmall, 0><<<lb, kBkThreads, sizeof(LsSmem<kLsCapSmall>), st>>>(
+        s.k[1], s.v[1], s.offset, nb, shift, flag);
+    count_launches(1);
+    // buckets above the small capacity (skewed keys): one block per SM, 200 KB shared memory
+    unsigned lb2 = (unsigned)nb < (unsigned)num_sms ? (unsigned)nb : (unsigned)num_sms;
+    bucket_local_sort_kernel<kLsCapLarge, kLsCapSmall><<<lb2, kBkThreads, sizeof(LsSmem<kLsCapLarge>), st>>>(
+        s.k[1], s.v[1], s.offset, nb, shift, flag);
     count_launches(1);
 }
 
