@@ -224,29 +224,58 @@ class _DevArray:
 class Result:
     """A query result. ``columns``: name -> numpy array (zero-copy view of library-owned pinned
     memory, valid until h2tap_free) or, for device results, a __cuda_array_interface__ object.
-    ``nulls``: name -> uint8 array, only for columns that can hold NULL."""
+    ``nulls``: name -> uint8 array, only for columns that can hold NULL. Columns, nulls and the
+    per-kernel times are materialised on first access (the scalar fields are read eagerly)."""
 
     def __init__(self, ptr):
         self._ptr = ptr
         r = ptr.contents
         self.epoch, self.nrows, self.on_device = r.epoch, r.nrows, bool(r.on_device)
         self.rows_scanned, self.device_ms, self.e2e_ms = r.rows_scanned, r.device_ms, r.e2e_ms
-        self.columns, self.nulls = {}, {}
+        self.kernel_launches = r.kernel_launches
+        self.plan_flags = r.plan_flags
+        self._columns = self._nulls = self._kernels = None
+
+    def _materialise(self):
+        r = self._ptr.contents
+        cols, nulls = {}, {}
         for i in range(r.ncols):
             name = r.names[i].decode()
             dt = _DT[r.types[i]]
             p = r.cols[i]
             if self.on_device:
-                self.columns[name] = _DevArray(p, self.nrows, dt)
+                cols[name] = _DevArray(p, self.nrows, dt)
             elif self.nrows:
-                self.columns[name] = np.ctypeslib.as_array(C.cast(p, C.POINTER(np.ctypeslib.as_ctypes_type(dt))), (self.nrows,))
+                cols[name] = np.ctypeslib.as_array(C.cast(p, C.POINTER(np.ctypeslib.as_ctypes_type(dt))), (self.nrows,))
             else:
-                self.columns[name] = np.zeros(0, dt)
+                cols[name] = np.zeros(0, dt)
             if bool(r.nulls[i]):
-                self.nulls[name] = np.ctypeslib.as_array(r.nulls[i], (self.nrows,)).copy()
-        self.kernel_launches = r.kernel_launches
-        self.plan_flags = r.plan_flags
-        self.kernels = [(r.kernel_names[i].decode(), r.kernel_ms[i]) for i in range(r.nkernels)]
+                nulls[name] = np.ctypeslib.as_array(r.nulls[i], (self.nrows,)).copy()
+        self._columns, self._nulls = cols, nulls
+
+    @property
+    def columns(self):
+        if self._columns is None:
+            if not self._ptr:
+                return {}
+            self._materialise()
+        return self._columns
+
+    @property
+    def nulls(self):
+        if self._nulls is None:
+            if not self._ptr:
+                return {}
+            self._materialise()
+        return self._nulls
+
+    @property
+    def kernels(self):
+        """[(kernel name, CUDA-event ms)] recorded with H2TAP_QUERY_PROFILE."""
+        if self._kernels is None:
+            r = self._ptr.contents
+            self._kernels = [(r.kernel_names[i].decode(), r.kernel_ms[i]) for i in range(r.nkernels)]
+        return self._kernels
 
     def to_numpy(self) -> dict:
         """Copy every column to a fresh host numpy array (device results via torch)."""
@@ -274,7 +303,7 @@ def h2tap_free(result: Result) -> None:
     if result is not None and result._ptr:
         _lib.h2tap_free(result._ptr)
         result._ptr = None
-        result.columns = {}
+        result._columns = {}
 
 
 def h2tap_compute_stream(engine: Engine) -> int:

@@ -866,6 +866,7 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
         bs.count = static_cast<unsigned int *>(e->arena.get("q18.bcount", 4 * ((1 << kBucketMaxBits) + 1)));
         bs.cursor = static_cast<unsigned int *>(e->arena.get("q18.bcursor", 4 * (1 << kBucketMaxBits)));
         bs.offset = static_cast<unsigned int *>(e->arena.get("q18.boffset", 4 * ((1 << kBucketMaxBits) + 1)));
+        bs.big = static_cast<unsigned int *>(e->arena.get("q18.bbig", 4 * ((1 << kBucketMaxBits) + 1)));
         int bb = 1;
         while (bb < kBucketMaxBits && (nout >> (bb + 9)) > 0) ++bb;   // ~256-512 rows per bucket
         e->prof.run("q18_sort_keys", [&] { launch_q18_sort_keys(rows, amt, nout, sp, sp2, e->num_sms, e->compute); });
@@ -986,6 +987,9 @@ h2tap_status query_impl(h2tap_engine *e, uint32_t plan, const int64_t *params, u
     if (!v) return fail(H2TAP_EPLAN, "no snapshot has been published yet");
     std::unique_ptr<ResultImpl> r(new_result(e, *v, flags & H2TAP_RESULT_DEVICE));
     e->prof.reset(flags & H2TAP_QUERY_PROFILE, e->compute);
+    // with per-kernel profiling, a short gate lets the whole query be enqueued before the GPU
+    // starts it, so no kernel's event window contains host launch latency
+    if (flags & H2TAP_QUERY_PROFILE) launch_gate(30000, e->compute);
     const uint64_t launches0 = launches_total();
     CK(cudaEventRecord(e->q_begin, e->compute));
     switch (plan) {

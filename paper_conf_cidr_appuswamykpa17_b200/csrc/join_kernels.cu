@@ -163,17 +163,30 @@ q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ o
     const uint64_t gwarp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
     const uint64_t nvec = n >> 2;  // full 4-row groups; the ragged tail is handled below
-    for (uint64_t vb = gwarp * 32; vb < nvec; vb += nwarps * 32) {
+    const uint64_t step = nwarps * 32;
+    // software pipeline: the next iteration's five 128-bit loads are in flight while the current
+    // group's runs are summed, probed and accumulated
+    int4 nW = make_int4(0, 0, 0, 0), nD = nW, nO = nW;
+    longlong2 nA0 = make_longlong2(0, 0), nA1 = nA0;
+    auto load = [&](uint64_t v) {
+        if (v < nvec) {
+            nW = __ldcs(reinterpret_cast<const int4 *>(ol_w) + v);
+            nD = __ldcs(reinterpret_cast<const int4 *>(ol_d) + v);
+            nO = __ldcs(reinterpret_cast<const int4 *>(ol_o) + v);
+            nA0 = __ldcs(reinterpret_cast<const longlong2 *>(ol_amt) + 2 * v);
+            nA1 = __ldcs(reinterpret_cast<const longlong2 *>(ol_amt) + 2 * v + 1);
+        }
+    };
+    load(gwarp * 32 + lane);
+    for (uint64_t vb = gwarp * 32; vb < nvec; vb += step) {
         const uint64_t v = vb + lane;
         const bool valid = v < nvec;
+        const int4 W = nW, D = nD, O = nO;
+        const longlong2 A0 = nA0, A1 = nA1;
+        load(v + step);
         Key3 k[4];
         long long a[4];
         if (valid) {
-            const int4 W = __ldcs(reinterpret_cast<const int4 *>(ol_w) + v);
-            const int4 D = __ldcs(reinterpret_cast<const int4 *>(ol_d) + v);
-            const int4 O = __ldcs(reinterpret_cast<const int4 *>(ol_o) + v);
-            const longlong2 A0 = __ldcs(reinterpret_cast<const longlong2 *>(ol_amt) + 2 * v);
-            const longlong2 A1 = __ldcs(reinterpret_cast<const longlong2 *>(ol_amt) + 2 * v + 1);
             k[0] = {W.x, D.x, O.x}; k[1] = {W.y, D.y, O.y}; k[2] = {W.z, D.z, O.z}; k[3] = {W.w, D.w, O.w};
             a[0] = A0.x; a[1] = A0.y; a[2] = A1.x; a[3] = A1.y;
         } else {

@@ -132,6 +132,7 @@ struct BucketSort {
     unsigned int *count;   // [2^kBucketMaxBits + 1]
     unsigned int *cursor;  // [2^kBucketMaxBits]
     unsigned int *offset;  // [2^kBucketMaxBits + 1]
+    unsigned int *big;     // [1 + 2^kBucketMaxBits]: count, then ids of buckets > small capacity
 };
 // Sorted pairs end in k[1]/v[1] (input in k[0]/v[0]).
 void bucket_sort_pairs(uint64_t n, int bits, int bucket_bits, const BucketSort &s, unsigned int *flag,
@@ -163,7 +164,8 @@ void launch_q18_permute(const Q18Row *rows, const long long *amt, const unsigned
                         const Q18Cols &dst, int num_sms, cudaStream_t st);
 
 // ------------------------------------------------------------ store (a1) --
-void launch_stats_init(int *out, int n_pairs, cudaStream_t st);  // pairs of (INT_MAX, INT_MIN)
+void launch_stats_init(int *out, int n_pairs, cudaStream_t st);
+void launch_gate(unsigned long long ns, cudaStream_t st);  // profiling only  // pairs of (INT_MAX, INT_MIN)
 void launch_minmax_i32(const int32_t *p, uint64_t n, int *out, int num_sms, cudaStream_t st);
 
 // ---------------------------------------------------------------- helpers --

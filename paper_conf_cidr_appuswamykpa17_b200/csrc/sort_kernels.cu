@@ -377,49 +377,49 @@ bucket_hist_kernel(const unsigned long long *__restrict__ key, uint64_t n, int s
         if (h[i]) atomicAdd(count + i, h[i]);
 }
 
-// exclusive scan of nb bucket counts -> offset[] and cursor[]; max bucket size -> count[nb]
+// exclusive scan of nb (<= 32768) bucket counts -> offset[] and cursor[]; one pass: each of
+// 1024 threads owns nb/1024 contiguous counts (all loads issued first); max size -> count[nb]
 __global__ void __launch_bounds__(1024) bucket_scan_kernel(unsigned int *__restrict__ count, int nb,
                                                            unsigned int *__restrict__ offset,
                                                            unsigned int *__restrict__ cursor) {
-    __shared__ unsigned int wsum[32];
-    __shared__ unsigned int carry_s;
+    __shared__ unsigned int wsum[32], wmax[32];
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    unsigned int carry = 0, mx = 0;
-    for (int r0 = 0; r0 < nb; r0 += 1024) {
-        const int i = r0 + threadIdx.x;
-        const unsigned int v = i < nb ? count[i] : 0u;
-        mx = max(mx, v);
-        unsigned int x = v;
+    const int per = (nb + 1023) / 1024;  // <= 32
+    const int b0 = threadIdx.x * per;
+    unsigned int t = 0, mx = 0;
+#pragma unroll 8
+    for (int q = 0; q < per; ++q) {  // pass 1: chunk total (re-read in pass 2 from L2)
+        const unsigned int c = b0 + q < nb ? count[b0 + q] : 0u;
+        t += c;
+        mx = max(mx, c);
+    }
+    unsigned int x = t;
 #pragma unroll
-        for (int o = 1; o < 32; o <<= 1) {
-            const unsigned int t = __shfl_up_sync(kFull, x, o);
-            if (lane >= o) x += t;
-        }
-        if (lane == 31) wsum[warp] = x;
-        __syncthreads();
-        if (warp == 0) {
-            unsigned int y = wsum[lane];
-#pragma unroll
-            for (int o = 1; o < 32; o <<= 1) {
-                const unsigned int t = __shfl_up_sync(kFull, y, o);
-                if (lane >= o) y += t;
-            }
-            wsum[lane] = y;
-            if (lane == 31) carry_s = y;
-        }
-        __syncthreads();
-        const unsigned int ex = carry + (warp ? wsum[warp - 1] : 0u) + x - v;
-        if (i < nb) { offset[i] = ex; cursor[i] = ex; }
-        carry += carry_s;
-        __syncthreads();
+    for (int o = 1; o < 32; o <<= 1) {
+        const unsigned int y = __shfl_up_sync(kFull, x, o);
+        if (lane >= o) x += y;
     }
     mx = __reduce_max_sync(kFull, mx);
-    if (lane == 0) wsum[warp] = mx;
+    if (lane == 31) wsum[warp] = x;
+    if (lane == 0) wmax[warp] = mx;
     __syncthreads();
+    unsigned int before = 0, total = 0, m = 0;
+    for (int w = 0; w < 32; ++w) {
+        before += w < warp ? wsum[w] : 0u;
+        total += wsum[w];
+        m = max(m, wmax[w]);
+    }
+    unsigned int run = before + x - t;
+#pragma unroll 8
+    for (int q = 0; q < per; ++q) {
+        if (b0 + q >= nb) break;
+        const unsigned int c = count[b0 + q];
+        offset[b0 + q] = run;
+        cursor[b0 + q] = run;
+        run += c;
+    }
     if (threadIdx.x == 0) {
-        unsigned int m = 0;
-        for (int w = 0; w < 32; ++w) m = max(m, wsum[w]);
-        offset[nb] = carry;
+        offset[nb] = total;
         count[nb] = m;
     }
 }
@@ -433,11 +433,12 @@ bucket_scatter_kernel(const unsigned long long *__restrict__ kin, const unsigned
     for (int i = threadIdx.x; i < nb; i += kBkThreads) h[i] = 0;
     const uint64_t base = (uint64_t)blockIdx.x * kBkThreads * kBkItems;
     unsigned long long k[kBkItems];
-    unsigned int b[kBkItems];
+    unsigned int b[kBkItems], val[kBkItems];
 #pragma unroll
     for (int i = 0; i < kBkItems; ++i) {
         const uint64_t j = base + (uint64_t)i * kBkThreads + threadIdx.x;
         k[i] = j < n ? __ldcs(kin + j) : 0ull;
+        val[i] = j < n ? __ldcs(vin + j) : 0u;
         b[i] = j < n ? (unsigned int)(k[i] >> shift) : 0xffffffffu;
     }
     __syncthreads();
@@ -449,13 +450,15 @@ bucket_scatter_kernel(const unsigned long long *__restrict__ kin, const unsigned
     for (int i = threadIdx.x; i < nb; i += kBkThreads)  // independent atomics: keep 8 in flight
         if (h[i]) h[i] = atomicAdd(cursor + i, h[i]);  // base of this block's range in bucket i
     __syncthreads();
+    unsigned int pos[kBkItems];
+#pragma unroll
+    for (int i = 0; i < kBkItems; ++i)
+        pos[i] = b[i] != 0xffffffffu ? atomicAdd(&h[b[i]], 1u) : 0u;
 #pragma unroll
     for (int i = 0; i < kBkItems; ++i) {
         if (b[i] == 0xffffffffu) continue;
-        const uint64_t j = base + (uint64_t)i * kBkThreads + threadIdx.x;
-        const unsigned int p = atomicAdd(&h[b[i]], 1u);
-        kout[p] = k[i];
-        vout[p] = __ldcs(vin + j);
+        kout[pos[i]] = k[i];
+        vout[pos[i]] = val[i];
     }
 }
 
@@ -474,15 +477,22 @@ template <int kLsCap, int kMin>
 __global__ void __launch_bounds__(kBkThreads)
 bucket_local_sort_kernel(unsigned long long *__restrict__ k, unsigned int *__restrict__ v,
                          const unsigned int *__restrict__ offset, int nb, int shift,
-                         unsigned int *flag) {
+                         unsigned int *flag, unsigned int *big) {
     extern __shared__ __align__(16) unsigned char smem_raw[];
     LsSmem<kLsCap> &S = *reinterpret_cast<LsSmem<kLsCap> *>(smem_raw);
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    for (int b = blockIdx.x; b < nb; b += gridDim.x) {
+    // the small instance walks every bucket and queues the big ones in big[1..]; the large
+    // instance walks only that queue
+    const int nwork = kMin > 0 ? (int)*(volatile unsigned int *)big : nb;
+    for (int wi = blockIdx.x; wi < nwork; wi += gridDim.x) {
+        const int b = kMin > 0 ? (int)big[1 + wi] : wi;
         const unsigned int lo = offset[b], m = offset[b + 1] - lo;
-        if (m <= (unsigned)(kMin > 1 ? kMin : 1)) continue;
+        if (m <= 1) continue;
         if (m > (unsigned)kLsCap) {
-            if (threadIdx.x == 0 && kMin > 0) atomicOr(flag, 2u);  // only the large instance flags
+            if (threadIdx.x == 0) {
+                if (kMin > 0) atomicOr(flag, 2u);                 // too big even for shared memory
+                else big[1 + atomicAdd(big, 1u)] = (unsigned)b;   // hand over to the large instance
+            }
             continue;
         }
         // sub-bucket bits: ~8 rows per sub-bucket, at most kLsSubMax sub-buckets
@@ -573,6 +583,7 @@ void bucket_sort_pairs(uint64_t n, int bits, int bucket_bits, const BucketSort &
         init = true;
     }
     cudaMemsetAsync(s.count, 0, sizeof(unsigned int) * (nb + 1), st);
+    cudaMemsetAsync(s.big, 0, sizeof(unsigned int), st);
     const uint64_t per = (uint64_t)kBkThreads * kBkItems;
     uint64_t hb = (n + per - 1) / per;
     if (hb > (uint64_t)num_sms * 2) hb = (uint64_t)num_sms * 2;
@@ -587,12 +598,12 @@ void bucket_sort_pairs(uint64_t n, int bits, int bucket_bits, const BucketSort &
     count_launches(1);
     unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
     bucket_local_sort_kernel<kLsCapSmall, 0><<<lb, kBkThreads, sizeof(LsSmem<kLsCapSmall>), st>>>(
-        s.k[1], s.v[1], s.offset, nb, shift, flag);
+        s.k[1], s.v[1], s.offset, nb, shift, flag, s.big);
     count_launches(1);
-    // buckets above the small capacity (skewed keys): one block per SM, 200 KB shared memory
-    unsigned lb2 = (unsigned)nb < (unsigned)num_sms ? (unsigned)nb : (unsigned)num_sms;
-    bucket_local_sort_kernel<kLsCapLarge, kLsCapSmall><<<lb2, kBkThreads, sizeof(LsSmem<kLsCapLarge>), st>>>(
-        s.k[1], s.v[1], s.offset, nb, shift, flag);
+    // buckets above the small capacity (skewed keys): one block per SM, ~200 KB shared memory
+    bucket_local_sort_kernel<kLsCapLarge, kLsCapSmall><<<(unsigned)num_sms, kBkThreads,
+                                                          sizeof(LsSmem<kLsCapLarge>), st>>>(
+        s.k[1], s.v[1], s.offset, nb, shift, flag, s.big);
     count_launches(1);
 }
 

@@ -33,7 +33,21 @@ __global__ void __launch_bounds__(256) minmax_kernel(const int32_t *__restrict__
     }
 }
 
+// Profiling gate: holds the stream for `ns` nanoseconds so the host can enqueue a query's
+// kernels behind it; per-kernel CUDA events then bracket only GPU execution, not host launch
+// latency (used with H2TAP_QUERY_PROFILE only).
+__global__ void gate_kernel(unsigned long long ns) {
+    unsigned long long t0, t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t0));
+    do {
+        __nanosleep(1000);
+        asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    } while (t - t0 < ns);
+}
+
 }  // namespace
+
+void launch_gate(unsigned long long ns, cudaStream_t st) { gate_kernel<<<1, 1, 0, st>>>(ns); }
 
 void launch_stats_init(int *out, int n_pairs, cudaStream_t st) {
     stats_init_kernel<<<(n_pairs + 127) / 128, 128, 0, st>>>(out, n_pairs);

@@ -1,4 +1,4 @@
-# ncu evidence for one round: launch list (cold, serialised) + one full capture per hot kernel.
+# ncu evidence for one round: launch list (cold, serialised) + one full capture of every hot kernel.
 # usage: bash scripts/ncu_round.sh <tag>
 set -x
 TAG=${1:-r01}
@@ -6,7 +6,6 @@ mkdir -p gpurun_out
 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/launches_${TAG}.csv \
     python scripts/profile_run.py --warehouses 100 --reps 2 > gpurun_out/launches_${TAG}.log 2>&1
 ncu --set full --clock-control none --import-source on \
-    -k regex:'q6_kernel|q1_kernel|q18_probe|q18_build|q18_having|scatter_kernel|hist_kernel|permute|q18_init' \
-    -c 12 -o gpurun_out/prof_${TAG} -f \
+    -k regex:'q6_kernel|q1_kernel|q18_|bucket_|sort_keys|tiefix|permute' \
+    -c 20 -o gpurun_out/prof_${TAG} -f \
     python scripts/profile_run.py --warehouses 100 --reps 1 > gpurun_out/prof_${TAG}.log 2>&1
-ls -la gpurun_out

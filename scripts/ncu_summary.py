@@ -53,4 +53,20 @@ open(md, "w").write(f"# ncu summary {tag}\n\n" + "\n".join(out) + "\n")
 print(open(md).read())
 if traffic:
     tj = os.path.join(root, "profiles", f"{tag}_traffic.json")
-    json.dump({k: sum(v) / len(v) for k, v in traffic.items()}, open(tj, "w"), indent=1)
+    per = {k: sum(v) / len(v) for k, v in traffic.items()}
+    json.dump(per, open(tj, "w"), indent=1)
+    # per-launch DRAM bytes keyed by the engine's profile marks (what bench.py reports)
+    marks = {"q6_kernel": "q6_scan_filter_sum", "q1_kernel": "q1_scan_filter_groupby",
+             "q18_init_kernel": "q18_init", "q18_build_kernel": "q18_build",
+             "q18_probe_kernel": "q18_probe_groupjoin", "q18_having_kernel": "q18_having_compact",
+             "sort_keys_kernel": "q18_sort_keys", "tiefix_kernel": "q18_tiefix",
+             "permute_kernel": "q18_permute"}
+    bymark = {}
+    for k, v in per.items():
+        m = marks.get(k, "q18_bucket_sort" if k.startswith("bucket_") else None)
+        if m:
+            bymark[m] = bymark.get(m, 0.0) + v
+    if len(sys.argv) > 2 and sys.argv[2] == "--bench":
+        json.dump({"source": f"profiles/{tag}_ncu_summary.md (ncu --set full, per launch)",
+                   **{k: int(v) for k, v in bymark.items()}},
+                  open(os.path.join(root, "profiles", "ncu_traffic.json"), "w"), indent=1)
