@@ -72,6 +72,11 @@ class h2tap_config(C.Structure):
                 ("nccl_unique_id", C.c_void_p)]
 
 
+class h2tap_query(C.Structure):
+    _fields_ = [("plan_id", C.c_uint32), ("nparams", C.c_uint32), ("params", C.POINTER(C.c_int64)),
+                ("flags", C.c_uint32)]
+
+
 class h2tap_result(C.Structure):
     _fields_ = [("epoch", C.c_uint64), ("nrows", C.c_uint64), ("ncols", C.c_uint32),
                 ("on_device", C.c_uint32), ("names", C.POINTER(C.c_char_p)),
@@ -91,6 +96,8 @@ _lib.h2tap_run_query_ex.argtypes = [_P, C.c_uint32, C.POINTER(C.c_int64), C.c_ui
                                     C.POINTER(C.POINTER(h2tap_result))]
 _lib.h2tap_run_query.argtypes = [_P, C.c_uint32, C.POINTER(C.c_int64), C.c_uint32,
                                  C.POINTER(C.POINTER(h2tap_result))]
+_lib.h2tap_run_queries.argtypes = [_P, C.POINTER(h2tap_query), C.c_uint32,
+                                   C.POINTER(C.POINTER(h2tap_result))]
 _lib.h2tap_free.argtypes = [C.POINTER(h2tap_result)]
 _lib.h2tap_free.restype = None
 _lib.h2tap_close.argtypes = [_P]
@@ -100,11 +107,12 @@ _lib.h2tap_nccl_unique_id.argtypes = [_P]
 _lib.h2tap_compute_stream.argtypes = [_P, C.POINTER(_P)]
 _lib.h2tap_c_last_name.argtypes = [C.c_int32, C.c_char_p, C.c_size_t]
 for _f in ("h2tap_open", "h2tap_load_snapshot_ex", "h2tap_load_snapshot", "h2tap_sync",
-           "h2tap_run_query_ex", "h2tap_run_query", "h2tap_nccl_unique_id", "h2tap_compute_stream"):
+           "h2tap_run_query_ex", "h2tap_run_query", "h2tap_run_queries", "h2tap_nccl_unique_id",
+           "h2tap_compute_stream"):
     getattr(_lib, _f).restype = C.c_int
 
 ABI_SYMBOLS = ["h2tap_open", "h2tap_load_snapshot", "h2tap_load_snapshot_ex", "h2tap_sync",
-               "h2tap_run_query", "h2tap_run_query_ex", "h2tap_free", "h2tap_close",
+               "h2tap_run_query", "h2tap_run_query_ex", "h2tap_run_queries", "h2tap_free", "h2tap_close",
                "h2tap_last_error", "h2tap_nccl_unique_id", "h2tap_compute_stream",
                "h2tap_c_last_name"]
 
@@ -297,6 +305,22 @@ def h2tap_run_query(engine: Engine, plan: int, params=None, *, flags: int = 0) -
     out = C.POINTER(h2tap_result)()
     _check(_lib.h2tap_run_query_ex(engine.handle, plan, parr, len(params), flags, C.byref(out)))
     return Result(out)
+
+
+def h2tap_run_queries(engine: Engine, queries) -> list:
+    """Run a batch on one published epoch: ``queries`` = [(plan, params or None, flags), ...].
+    All plans are enqueued back to back and the library synchronises once."""
+    n = len(queries)
+    qarr = (h2tap_query * max(1, n))()
+    keep = []
+    for i, (plan, params, flags) in enumerate(queries):
+        params = list(params or [])
+        parr = (C.c_int64 * max(1, len(params)))(*params)
+        keep.append(parr)
+        qarr[i] = h2tap_query(plan, len(params), parr, flags)
+    outs = (C.POINTER(h2tap_result) * max(1, n))()
+    _check(_lib.h2tap_run_queries(engine.handle, qarr, n, outs))
+    return [Result(outs[i]) for i in range(n)]
 
 
 def h2tap_free(result: Result) -> None:

@@ -549,8 +549,57 @@ void add_col(ResultImpl *r, const char *name, uint32_t type, const void *p) {
 
 void sync_compute(h2tap_engine *e) { CK(cudaStreamSynchronize(e->compute)); }
 
+// ---- query execution: launch (asynchronous) + finish (after one stream synchronisation) ------
+// A query's kernels are enqueued by launch(); finish() runs after the host has synchronised
+// with the compute stream, reads the few scalars it needs (counts, flags), and completes the
+// result (host copies when requested). h2tap_run_queries launches a whole batch, synchronises
+// once and finishes every query, so the GPU runs the batch back to back (the paper's "several
+// OLAP queries share a snapshot", L555-559). With world > 1 a plan synchronises inside launch
+// where a collective needs host-side sizes.
+struct QueryCtx {
+    uint32_t plan = 0, flags = 0;
+    int64_t p[4] = {};
+    std::unique_ptr<ResultImpl> r;
+    cudaEvent_t begin = nullptr, end = nullptr;
+    uint64_t launches0 = 0, launches = 0;
+    std::pair<void *, size_t> small{};     // pinned scalars read back at finish
+    std::chrono::steady_clock::time_point t0;
+    size_t mark0 = 0, mark1 = 0;           // this query's profile marks [mark0, mark1)
+    // Q1
+    Q1Scratch q1{};
+    std::vector<std::pair<void *, size_t>> dev_blocks;  // per-query device output blocks
+    // Q18
+    Q18Scratch q18{};
+    Q18Plan *plan_dev = nullptr;
+    const Q18Row *rows = nullptr;
+    const long long *amt = nullptr;
+    const unsigned int *perm = nullptr;
+    const unsigned long long *perm_keys = nullptr;
+    SortPairs sp{};
+    Q18Cols out{};                          // device output columns (sorted)
+    uint64_t n_max = 0;
+    unsigned int *tie_dev = nullptr;
+    bool q18_sorted_on_host_sync = false;   // world > 1 path already knows nout
+    uint64_t nout_host = 0;
+};
+
+void *dev_block(h2tap_engine *e, QueryCtx &q, size_t bytes) {
+    auto b = e->dev_pool->get(bytes ? bytes : 8);
+    q.dev_blocks.push_back(b);
+    return b.first;
+}
+void release_dev_blocks(h2tap_engine *e, QueryCtx &q) {
+    for (auto &b : q.dev_blocks) e->dev_pool->put(b.first, b.second);
+    q.dev_blocks.clear();
+}
+// Device output blocks become the result's columns (ownership moves to the result).
+void give_blocks_to_result(QueryCtx &q) {
+    for (auto &b : q.dev_blocks) q.r->blocks.push_back(b);
+    q.dev_blocks.clear();
+}
+
 // ---- Q6 (a2 + a7)
-void run_q6(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
+void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     const int T = H2TAP_T_ORDER_LINE;
     need_cols(v, T, {H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}, "Q6");
     Q6Scratch s;
@@ -560,7 +609,7 @@ void run_q6(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
     s.out = static_cast<long long *>(e->arena.get("q6.out", 64));
     e->prof.run("q6_scan_filter_sum", [&] {
         launch_q6(colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D), colp<int32_t>(v, T, H2TAP_OL_QUANTITY),
-                  colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T], p[0], p[1], p[2], p[3], s,
+                  colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T], q.p[0], q.p[1], q.p[2], q.p[3], s,
                   e->num_sms, e->compute);
         CK(cudaGetLastError());
     });
@@ -568,54 +617,52 @@ void run_q6(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
         e->prof.run("q6_allreduce", [&] {
             NK(ncclAllReduce(s.out, s.out, 2, ncclInt64, ncclSum, e->comm, e->compute));
         });
-    CK(cudaMemcpyAsync(e->small_host, s.out, 16, cudaMemcpyDeviceToHost, e->compute));
-    CK(cudaEventRecord(e->q_end, e->compute));
-    sync_compute(e);
-    const long long rev = e->small_host[0], cnt = e->small_host[1];
+    CK(cudaMemcpyAsync(q.small.first, s.out, 16, cudaMemcpyDeviceToHost, e->compute));
+}
+
+void finish_q6(h2tap_engine *e, QueryCtx &q) {
+    ResultImpl *r = q.r.get();
+    const long long *sm = static_cast<const long long *>(q.small.first);
+    const long long rev = sm[0], cnt = sm[1];
     r->nrows = 1;
     auto *blk = static_cast<long long *>(result_block(r, 16));
-    if (r->on_device) CK(cudaMemcpy(blk, e->small_host, 16, cudaMemcpyHostToDevice));
+    if (r->on_device) CK(cudaMemcpy(blk, sm, 16, cudaMemcpyHostToDevice));
     else { blk[0] = rev; blk[1] = cnt; }
+    (void)e;
     add_col(r, "revenue", H2TAP_I64, blk);
     r->null_store.back().assign(1, cnt == 0 ? 1 : 0);  // SUM over no rows IS NULL (R8)
     add_col(r, "count_rows", H2TAP_I64, blk + 1);
 }
 
 // ---- Q1 (a3 + a7 + a8)
-void run_q1(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
+constexpr size_t kQ1MaxGroups = kQ1GlobalSlots + kQ1Dense;
+
+void launch_q1_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     const int T = H2TAP_T_ORDER_LINE;
     need_cols(v, T, {H2TAP_OL_NUMBER, H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}, "Q1");
-    Q1Scratch s;
-    const size_t maxg = kQ1GlobalSlots + kQ1Dense;
-    bool fresh = !e->arena.bufs.count("q1.gtag");
+    Q1Scratch &s = q.q1;
+    const bool fresh = !e->arena.bufs.count("q1.gtag");
     s.dense = static_cast<unsigned long long *>(e->arena.get("q1.dense", 8 * kQ1Dense * 3));
     s.gtag = static_cast<unsigned long long *>(e->arena.get("q1.gtag", 8ull * kQ1GlobalSlots));
     s.gacc = static_cast<unsigned long long *>(e->arena.get("q1.gacc", 24ull * kQ1GlobalSlots));
     s.flags = static_cast<unsigned int *>(e->arena.get("q1.flags", 64));
-    s.groups = static_cast<Q1Group *>(e->arena.get("q1.groups", sizeof(Q1Group) * maxg));
+    s.groups = static_cast<Q1Group *>(e->arena.get("q1.groups", sizeof(Q1Group) * kQ1MaxGroups));
     s.ngroups = static_cast<unsigned long long *>(e->arena.get("q1.ngroups", 64));
-    s.o_key = static_cast<int32_t *>(e->arena.get("q1.okey", 4 * maxg));
-    s.o_qty = static_cast<long long *>(e->arena.get("q1.oqty", 8 * maxg));
-    s.o_amt = static_cast<long long *>(e->arena.get("q1.oamt", 8 * maxg));
-    s.o_cnt = static_cast<long long *>(e->arena.get("q1.ocnt", 8 * maxg));
-    s.o_avg_qty = static_cast<double *>(e->arena.get("q1.oavgq", 8 * maxg));
-    s.o_avg_amt = static_cast<double *>(e->arena.get("q1.oavga", 8 * maxg));
+    // outputs go straight into per-query device blocks (they become the result's columns)
+    s.o_key = static_cast<int32_t *>(dev_block(e, q, 4 * kQ1MaxGroups));
+    s.o_qty = static_cast<long long *>(dev_block(e, q, 8 * kQ1MaxGroups));
+    s.o_amt = static_cast<long long *>(dev_block(e, q, 8 * kQ1MaxGroups));
+    s.o_avg_qty = static_cast<double *>(dev_block(e, q, 8 * kQ1MaxGroups));
+    s.o_avg_amt = static_cast<double *>(dev_block(e, q, 8 * kQ1MaxGroups));
+    s.o_cnt = static_cast<long long *>(dev_block(e, q, 8 * kQ1MaxGroups));
     if (fresh) launch_q1_reset(s, e->compute);  // tables self-clean afterwards (q1_compact)
     e->prof.run("q1_scan_filter_groupby", [&] {
         launch_q1(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
                   colp<int32_t>(v, T, H2TAP_OL_QUANTITY), colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T],
-                  p[0], s, e->num_sms, e->compute);
+                  q.p[0], s, e->num_sms, e->compute);
         CK(cudaGetLastError());
     });
     e->prof.run("q1_compact", [&] { launch_q1_compact(s, e->compute); });
-    CK(cudaMemcpyAsync(e->small_host, s.ngroups, 8, cudaMemcpyDeviceToHost, e->compute));
-    CK(cudaMemcpyAsync(e->small_host + 1, s.flags, 4, cudaMemcpyDeviceToHost, e->compute));
-    sync_compute(e);
-    uint64_t ng = (uint64_t)e->small_host[0];
-    if (e->small_host[1] & 1) {
-        CK(cudaMemsetAsync(s.flags, 0, 4, e->compute));
-        raise(H2TAP_ENOMEM, "Q1: more than %d distinct ol_number groups", kQ1GlobalSlots);
-    }
     if (e->world > 1) {  // a7: gather every rank's groups, fold into one table, re-compact
         auto *cnt_dev = static_cast<unsigned long long *>(e->arena.get("q1.allcnt", 8ull * e->world));
         e->prof.run("q1_allgather", [&] {
@@ -635,45 +682,43 @@ void run_q1(h2tap_engine *e, const View &v, const int64_t *p, ResultImpl *r) {
                 if (cnts[k]) launch_q1_merge(all + (uint64_t)k * gcap, cnts[k], s, e->compute);
             launch_q1_compact(s, e->compute);
         });
-        CK(cudaMemcpyAsync(e->small_host, s.ngroups, 8, cudaMemcpyDeviceToHost, e->compute));
-        sync_compute(e);
-        ng = (uint64_t)e->small_host[0];
     }
-    e->prof.run("q1_emit", [&] { launch_q1_emit(s, ng, e->compute); });
+    e->prof.run("q1_emit", [&] { launch_q1_emit(s, kQ1MaxGroups, e->compute); });
+    auto *sm = static_cast<unsigned long long *>(q.small.first);
+    CK(cudaMemcpyAsync(sm, s.ngroups, 8, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaMemcpyAsync(sm + 1, s.flags, 4, cudaMemcpyDeviceToHost, e->compute));
+}
+
+void finish_q1(h2tap_engine *e, QueryCtx &q) {
+    ResultImpl *r = q.r.get();
+    const auto *sm = static_cast<const unsigned long long *>(q.small.first);
+    const uint64_t ng = sm[0];
+    if (static_cast<const unsigned int *>(q.small.first)[2] & 1) {
+        CK(cudaMemsetAsync(q.q1.flags, 0, 4, e->compute));
+        raise(H2TAP_ENOMEM, "Q1: more than %d distinct ol_number groups", kQ1GlobalSlots);
+    }
     r->nrows = ng;
+    const Q1Scratch &s = q.q1;
     struct { const char *name; uint32_t type; const void *src; size_t es; } cols[] = {
         {"ol_number", H2TAP_I32, s.o_key, 4}, {"sum_qty", H2TAP_I64, s.o_qty, 8},
         {"sum_amount", H2TAP_I64, s.o_amt, 8}, {"avg_qty", H2TAP_F64, s.o_avg_qty, 8},
         {"avg_amount", H2TAP_F64, s.o_avg_amt, 8}, {"count_order", H2TAP_I64, s.o_cnt, 8}};
+    if (r->on_device) {
+        for (auto &c : cols) add_col(r, c.name, c.type, c.src);
+        give_blocks_to_result(q);
+        return;
+    }
     for (auto &c : cols) {
         void *dst = result_block(r, ng * c.es);
-        if (ng)
-            CK(cudaMemcpyAsync(dst, c.src, ng * c.es,
-                               r->on_device ? cudaMemcpyDeviceToDevice : cudaMemcpyDeviceToHost,
-                               e->compute));
+        if (ng) CK(cudaMemcpyAsync(dst, c.src, ng * c.es, cudaMemcpyDeviceToHost, e->compute));
         add_col(r, c.name, c.type, dst);
     }
-    CK(cudaEventRecord(e->q_end, e->compute));
     sync_compute(e);
+    release_dev_blocks(e, q);
 }
 
 // ---- Q18 (a4 + a5 + a6 + a7 + a8)
 int bitwidth(unsigned long long x) { return x ? 64 - __builtin_clzll(x) : 0; }
-
-Q18Cols carve_cols(Arena &a, const char *prefix, uint64_t n) {
-    auto nm = [&](const char *c) { return std::string(prefix) + c; };
-    const uint64_t m = std::max<uint64_t>(n, 1);
-    Q18Cols c;
-    c.c_last = static_cast<int32_t *>(a.get(nm("c_last"), 4 * m));
-    c.c_id = static_cast<int32_t *>(a.get(nm("c_id"), 4 * m));
-    c.o_id = static_cast<int32_t *>(a.get(nm("o_id"), 4 * m));
-    c.o_ol_cnt = static_cast<int32_t *>(a.get(nm("o_ol_cnt"), 4 * m));
-    c.o_w_id = static_cast<int32_t *>(a.get(nm("o_w_id"), 4 * m));
-    c.o_d_id = static_cast<int32_t *>(a.get(nm("o_d_id"), 4 * m));
-    c.o_entry_d = static_cast<int64_t *>(a.get(nm("o_entry_d"), 8 * m));
-    c.amount_sum = static_cast<int64_t *>(a.get(nm("amount_sum"), 8 * m));
-    return c;
-}
 
 uint64_t pow2_at_least(uint64_t x) {
     uint64_t c = 16;
@@ -711,14 +756,66 @@ JoinIndex plan_index(h2tap_engine *e, const View &v, int table, bool force_hash,
     return j;
 }
 
-void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, ResultImpl *r) {
+struct Q18Small { unsigned long long nout; unsigned int err, tie; Q18Stats st; };
+
+void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
+    // a8: ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id, entirely on the device:
+    // plan (field widths from the stats) -> 64-bit prefix keys -> bucket sort -> tie-fix ->
+    // gather into the output columns. Grids are sized for n_max (the orders rows).
+    const uint64_t n_max = std::max<uint64_t>(q.n_max, 1);
+    int bb = 1;
+    while (bb < kBucketMaxBits && (n_max >> (bb + 9)) > 0) ++bb;   // ~256-512 rows per bucket
+    q.plan_dev = static_cast<Q18Plan *>(e->arena.get("q18.plan", sizeof(Q18Plan)));
+    e->prof.run("q18_plan", [&] { launch_q18_plan(q.q18.stats, q.q18.nout, bb, q.plan_dev, e->compute); });
+    for (int b = 0; b < 2; ++b) {
+        q.sp.k[b] = static_cast<unsigned long long *>(e->arena.get("q18.sk" + std::to_string(b), 8 * n_max));
+        q.sp.v[b] = static_cast<unsigned int *>(e->arena.get("q18.sv" + std::to_string(b), 4 * n_max));
+    }
+    q.sp.counts = static_cast<unsigned int *>(e->arena.get("q18.counts", 4ull * 256 * sort_tiles(n_max)));
+    q.sp.totals = static_cast<unsigned int *>(e->arena.get("q18.totals", 4 * 256));
+    BucketSort bs;
+    bs.k[0] = q.sp.k[0]; bs.k[1] = q.sp.k[1]; bs.v[0] = q.sp.v[0]; bs.v[1] = q.sp.v[1];
+    bs.count = static_cast<unsigned int *>(e->arena.get("q18.bcount", 4 * ((1 << kBucketMaxBits) + 1)));
+    bs.cursor = static_cast<unsigned int *>(e->arena.get("q18.bcursor", 4 * (1 << kBucketMaxBits)));
+    bs.offset = static_cast<unsigned int *>(e->arena.get("q18.boffset", 4 * ((1 << kBucketMaxBits) + 1)));
+    bs.big = static_cast<unsigned int *>(e->arena.get("q18.bbig", 4 * ((1 << kBucketMaxBits) + 1)));
+    q.tie_dev = static_cast<unsigned int *>(e->arena.get("q18.tie", 64));
+    CK(cudaMemsetAsync(q.tie_dev, 0, 4, e->compute));
+    e->prof.run("q18_sort_keys", [&] {
+        launch_q18_sort_keys(q.rows, q.amt, q.plan_dev, n_max, q.sp, e->num_sms, e->compute);
+    });
+    e->prof.run("q18_bucket_sort", [&] {
+        bucket_sort_pairs(n_max, &q.plan_dev->n, &q.plan_dev->shift, bb, bs, q.tie_dev, e->num_sms,
+                          e->compute);
+    });
+    e->prof.run("q18_tiefix", [&] {
+        launch_q18_tiefix(q.rows, q.amt, q.sp.k[1], q.sp.v[1], q.plan_dev, n_max, q.tie_dev,
+                          e->num_sms, e->compute);
+    });
+    q.perm = q.sp.v[1];
+    q.perm_keys = q.sp.k[1];
+    Q18Cols &d = q.out;
+    d.c_last = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    d.c_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    d.o_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    d.o_entry_d = static_cast<int64_t *>(dev_block(e, q, 8 * n_max));
+    d.o_ol_cnt = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    d.amount_sum = static_cast<int64_t *>(dev_block(e, q, 8 * n_max));
+    d.o_w_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    d.o_d_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    e->prof.run("q18_permute", [&] {
+        launch_q18_permute(q.rows, q.amt, q.perm, q.perm_keys, q.plan_dev, n_max, d, e->num_sms, e->compute);
+    });
+}
+
+void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
     need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}, "Q18");
     need_cols(v, O, {H2TAP_O_W_ID, H2TAP_O_D_ID, H2TAP_O_ID, H2TAP_O_C_ID, H2TAP_O_OL_CNT, H2TAP_O_ENTRY_D}, "Q18");
     need_cols(v, C, {H2TAP_C_W_ID, H2TAP_C_D_ID, H2TAP_C_ID, H2TAP_C_LAST}, "Q18");
     const uint64_t n_ol = v.n[OL], n_o = v.n[O], n_c = v.n[C];
-    const bool force_hash = flags & H2TAP_QUERY_HASH_JOIN;
-    Q18Scratch s;
+    const bool force_hash = q.flags & H2TAP_QUERY_HASH_JOIN;
+    Q18Scratch &s = q.q18;
     s.jo = plan_index(e, v, O, force_hash, "q18.jo");
     s.jc = plan_index(e, v, C, force_hash, "q18.jc");
     s.acc = static_cast<Q18Acc *>(e->arena.get("q18.acc", sizeof(Q18Acc) * std::max<uint64_t>(n_o, 1)));
@@ -729,7 +826,7 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
     s.ticket = static_cast<unsigned int *>(e->arena.get("q18.ticket", 64, true, e->compute));
     s.rows = static_cast<Q18Row *>(e->arena.get("q18.rows", sizeof(Q18Row) * std::max<uint64_t>(n_o, 1)));
     s.amt = static_cast<long long *>(e->arena.get("q18.amt", 8 * std::max<uint64_t>(n_o, 1)));
-    r->plan_flags = (s.jo.dense ? 1u : 0u) | (s.jc.dense ? 2u : 0u);
+    q.r->plan_flags = (s.jo.dense ? 1u : 0u) | (s.jc.dense ? 2u : 0u);
 
     e->prof.run("q18_init", [&] { launch_q18_init(s, n_o, e->num_sms, e->compute); });
     e->prof.run("q18_build", [&] {
@@ -749,36 +846,26 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
             launch_q18_having(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
                               colp<int32_t>(v, O, H2TAP_O_ID), colp<int32_t>(v, O, H2TAP_O_C_ID),
                               colp<int32_t>(v, O, H2TAP_O_OL_CNT), colp<int64_t>(v, O, H2TAP_O_ENTRY_D),
-                              n_o, colp<int32_t>(v, C, H2TAP_C_LAST), p[0], s, e->num_sms, e->compute);
+                              n_o, colp<int32_t>(v, C, H2TAP_C_LAST), q.p[0], s, e->num_sms, e->compute);
     });
     CK(cudaGetLastError());
-    // small D2H: err, nout, stats
-    struct Small { unsigned long long nout; unsigned int err, tie; Q18Stats st; };
-    static_assert(sizeof(Small) <= 256, "small");
-    Small *sm = reinterpret_cast<Small *>(e->small_host);
-    CK(cudaMemcpyAsync(&sm->nout, s.nout, 8, cudaMemcpyDeviceToHost, e->compute));
-    CK(cudaMemcpyAsync(&sm->err, s.err, 4, cudaMemcpyDeviceToHost, e->compute));
-    CK(cudaMemcpyAsync(&sm->st, s.stats, sizeof(Q18Stats), cudaMemcpyDeviceToHost, e->compute));
-    sync_compute(e);
-    const unsigned int err = sm->err;
-    uint64_t nout = sm->nout;
-    Q18Stats st = sm->st;
-    int err_any = err ? 1 : 0;
-    if (e->world > 1) {  // every rank must learn whether any rank failed before the next collective
+    q.rows = s.rows;
+    q.amt = s.amt;
+    q.n_max = n_o;
+    Q18Small *sm = static_cast<Q18Small *>(q.small.first);
+    if (e->world > 1) {
+        // a7: groups are warehouse-local; gather the result rows to rank 0 (host-sized NCCL calls)
+        CK(cudaMemcpyAsync(&sm->nout, s.nout, 8, cudaMemcpyDeviceToHost, e->compute));
+        CK(cudaMemcpyAsync(&sm->err, s.err, 4, cudaMemcpyDeviceToHost, e->compute));
+        sync_compute(e);
+        int err_any = sm->err ? 1 : 0;
         auto *flag = static_cast<int *>(e->arena.get("q18.errflag", 64));
         CK(cudaMemcpyAsync(flag, &err_any, 4, cudaMemcpyHostToDevice, e->compute));
         NK(ncclAllReduce(flag, flag, 1, ncclInt32, ncclMax, e->comm, e->compute));
         CK(cudaMemcpyAsync(&err_any, flag, 4, cudaMemcpyDeviceToHost, e->compute));
         sync_compute(e);
-    }
-    if (err & kErrDupOrders) raise(H2TAP_EDUPKEY, "Q18: duplicate orders primary key (w, d, o_id)");
-    if (err & kErrDupCustomer) raise(H2TAP_EDUPKEY, "Q18: duplicate customer primary key (w, d, c_id)");
-    if (err & kErrDomain) raise(H2TAP_EPLAN, "Q18: join key outside the supported domain");
-    if (err_any) raise(H2TAP_EPLAN, "Q18: failed on another rank");
-
-    const Q18Row *rows = s.rows;
-    const long long *amt = s.amt;
-    if (e->world > 1) {  // a7: groups are warehouse-local; gather result rows to rank 0
+        if (sm->err) return;  // finish raises the local error
+        if (err_any) raise(H2TAP_EPLAN, "Q18: failed on another rank");
         auto *cnt_dev = static_cast<unsigned long long *>(e->arena.get("q18.allcnt", 8ull * e->world));
         NK(ncclAllGather(s.nout, cnt_dev, 1, ncclUint64, e->comm, e->compute));
         std::vector<unsigned long long> cnts(e->world);
@@ -811,145 +898,74 @@ void run_q18(h2tap_engine *e, const View &v, const int64_t *p, uint32_t flags, R
             }
             NK(ncclGroupEnd());
         });
-        if (e->rank != 0) {
-            CK(cudaEventRecord(e->q_end, e->compute));
-            sync_compute(e);
-            r->nrows = 0;
-            const char *names[] = {"c_last", "c_id", "o_id", "o_entry_d", "o_ol_cnt", "amount_sum", "o_w_id", "o_d_id"};
-            const uint32_t types[] = {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I32};
-            for (int i = 0; i < 8; ++i) add_col(r, names[i], types[i], result_block(r, 8));
+        if (e->rank != 0) {  // rows are returned on rank 0 only
+            q.q18_sorted_on_host_sync = true;
+            q.nout_host = 0;
             return;
         }
-        nout = total;
-        rows = all;
-        amt = all_amt;
-        Q18Stats init;
-        init.amt_min = INT64_MAX; init.amt_max = INT64_MIN; init.ent_min = INT64_MAX; init.ent_max = INT64_MIN;
-        init.w_min = INT32_MAX; init.w_max = INT32_MIN; init.d_min = INT32_MAX; init.d_max = INT32_MIN;
-        init.o_min = INT32_MAX; init.o_max = INT32_MIN; init.pad0 = init.pad1 = 0;
-        sm->st = init;
-        CK(cudaMemcpyAsync(s.stats, &sm->st, sizeof(Q18Stats), cudaMemcpyHostToDevice, e->compute));
-        launch_q18_stats(rows, amt, nout, s, e->num_sms, e->compute);
-        CK(cudaMemcpyAsync(&sm->st, s.stats, sizeof(Q18Stats), cudaMemcpyDeviceToHost, e->compute));
-        sync_compute(e);
-        st = sm->st;
+        q.rows = all;
+        q.amt = all_amt;
+        q.n_max = total;
+        sm->nout = total;
+        CK(cudaMemcpyAsync(s.nout, &sm->nout, 8, cudaMemcpyHostToDevice, e->compute));
+        launch_q18_stats(all, all_amt, total, s, e->num_sms, e->compute);  // stats of gathered rows
     }
+    q18_sort_and_emit(e, q);
+    CK(cudaMemcpyAsync(&sm->nout, s.nout, 8, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaMemcpyAsync(&sm->err, s.err, 4, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaMemcpyAsync(&sm->tie, q.tie_dev, 4, cudaMemcpyDeviceToHost, e->compute));
+}
 
-    // a8: ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id — radix sort of row ids
-    Q18SortSpec sp{};
-    SortPairs sp2{};
-    const unsigned int *perm = nullptr;
-    const unsigned long long *perm_keys = nullptr;  // sorted prefix keys parallel to perm
-    unsigned int *tie_dev = static_cast<unsigned int *>(e->arena.get("q18.tie", 64));
-    bool tiefix = false;
-    if (nout > 1) {
-        sp.amt_max = st.amt_max;
-        sp.ent_min = st.ent_min;
-        sp.w_min = st.w_min; sp.d_min = st.d_min; sp.o_min = st.o_min;
-        sp.nd = (long long)st.d_max - st.d_min + 1;
-        sp.no = (long long)st.o_max - st.o_min + 1;
-        const unsigned long long nw = (unsigned long long)((long long)st.w_max - st.w_min + 1);
-        sp.bits_a = bitwidth((unsigned long long)st.amt_max - (unsigned long long)st.amt_min);
-        sp.bits_e = bitwidth((unsigned long long)st.ent_max - (unsigned long long)st.ent_min);
-        sp.bits_r = bitwidth(nw * (unsigned long long)sp.nd * (unsigned long long)sp.no - 1);
-        const int B = sp.bits_a + sp.bits_e + sp.bits_r;
-        sp.prefix_bits = B <= 64 ? B : 64;
-        tiefix = B > sp.prefix_bits;
-        for (int b = 0; b < 2; ++b) {
-            sp2.k[b] = static_cast<unsigned long long *>(e->arena.get("q18.sk" + std::to_string(b), 8 * nout));
-            sp2.v[b] = static_cast<unsigned int *>(e->arena.get("q18.sv" + std::to_string(b), 4 * nout));
-        }
-        sp2.counts = static_cast<unsigned int *>(e->arena.get("q18.counts", 4ull * 256 * sort_tiles(nout)));
-        sp2.totals = static_cast<unsigned int *>(e->arena.get("q18.totals", 4 * 256));
-        BucketSort bs;
-        bs.k[0] = sp2.k[0]; bs.k[1] = sp2.k[1]; bs.v[0] = sp2.v[0]; bs.v[1] = sp2.v[1];
-        bs.count = static_cast<unsigned int *>(e->arena.get("q18.bcount", 4 * ((1 << kBucketMaxBits) + 1)));
-        bs.cursor = static_cast<unsigned int *>(e->arena.get("q18.bcursor", 4 * (1 << kBucketMaxBits)));
-        bs.offset = static_cast<unsigned int *>(e->arena.get("q18.boffset", 4 * ((1 << kBucketMaxBits) + 1)));
-        bs.big = static_cast<unsigned int *>(e->arena.get("q18.bbig", 4 * ((1 << kBucketMaxBits) + 1)));
-        int bb = 1;
-        while (bb < kBucketMaxBits && (nout >> (bb + 9)) > 0) ++bb;   // ~256-512 rows per bucket
-        e->prof.run("q18_sort_keys", [&] { launch_q18_sort_keys(rows, amt, nout, sp, sp2, e->num_sms, e->compute); });
-        CK(cudaMemsetAsync(tie_dev, 0, 4, e->compute));
-        e->prof.run("q18_bucket_sort", [&] {
-            bucket_sort_pairs(nout, sp.prefix_bits, bb, bs, tie_dev, e->num_sms, e->compute);
-        });
-        perm = sp2.v[1];
-        perm_keys = sp2.k[1];
-        if (tiefix)
-            e->prof.run("q18_tiefix", [&] {
-                launch_q18_tiefix(rows, amt, sp2.k[1], sp2.v[1], nout, tie_dev, e->num_sms, e->compute);
-            });
-        tiefix = true;  // read the flag back: tie runs > 32 (bit 0) or a bucket > capacity (bit 1)
+void finish_q18(h2tap_engine *e, QueryCtx &q) {
+    ResultImpl *r = q.r.get();
+    Q18Small *sm = static_cast<Q18Small *>(q.small.first);
+    const char *names[] = {"c_last", "c_id", "o_id", "o_entry_d", "o_ol_cnt", "amount_sum", "o_w_id", "o_d_id"};
+    const uint32_t types[] = {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I32};
+    if (q.q18_sorted_on_host_sync) {  // world > 1, rank != 0
+        r->nrows = 0;
+        for (int i = 0; i < 8; ++i) add_col(r, names[i], types[i], result_block(r, 8));
+        release_dev_blocks(e, q);
+        return;
     }
-    r->nrows = nout;
-    Q18Cols dst;
-    auto alloc_dst = [&](bool device) {
-        auto blk = [&](size_t es) { return result_block(r, es * nout); };
-        if (device) {
-            dst.c_last = static_cast<int32_t *>(blk(4)); dst.c_id = static_cast<int32_t *>(blk(4));
-            dst.o_id = static_cast<int32_t *>(blk(4)); dst.o_entry_d = static_cast<int64_t *>(blk(8));
-            dst.o_ol_cnt = static_cast<int32_t *>(blk(4)); dst.amount_sum = static_cast<int64_t *>(blk(8));
-            dst.o_w_id = static_cast<int32_t *>(blk(4)); dst.o_d_id = static_cast<int32_t *>(blk(4));
-        }
-    };
-    Q18Cols host_dst{};
-    if (r->on_device) alloc_dst(true);
-    else {
-        dst = carve_cols(e->arena, "q18.sorted.", nout);
-        host_dst.c_last = static_cast<int32_t *>(result_block(r, 4 * nout));
-        host_dst.c_id = static_cast<int32_t *>(result_block(r, 4 * nout));
-        host_dst.o_id = static_cast<int32_t *>(result_block(r, 4 * nout));
-        host_dst.o_entry_d = static_cast<int64_t *>(result_block(r, 8 * nout));
-        host_dst.o_ol_cnt = static_cast<int32_t *>(result_block(r, 4 * nout));
-        host_dst.amount_sum = static_cast<int64_t *>(result_block(r, 8 * nout));
-        host_dst.o_w_id = static_cast<int32_t *>(result_block(r, 4 * nout));
-        host_dst.o_d_id = static_cast<int32_t *>(result_block(r, 4 * nout));
-    }
-    auto emit = [&]() {
-        e->prof.run("q18_permute", [&] {
-            if (nout) launch_q18_permute(rows, amt, perm, perm_keys, sp, nout, dst, e->num_sms, e->compute);
-        });
-        if (!r->on_device && nout) {
-            auto d2h = [&](void *h, const void *d, size_t es) {
-                CK(cudaMemcpyAsync(h, d, nout * es, cudaMemcpyDeviceToHost, e->compute));
-            };
-            d2h(host_dst.c_last, dst.c_last, 4); d2h(host_dst.c_id, dst.c_id, 4);
-            d2h(host_dst.o_id, dst.o_id, 4); d2h(host_dst.o_entry_d, dst.o_entry_d, 8);
-            d2h(host_dst.o_ol_cnt, dst.o_ol_cnt, 4); d2h(host_dst.amount_sum, dst.amount_sum, 8);
-            d2h(host_dst.o_w_id, dst.o_w_id, 4); d2h(host_dst.o_d_id, dst.o_d_id, 4);
-        }
-        if (tiefix) CK(cudaMemcpyAsync(&sm->tie, tie_dev, 4, cudaMemcpyDeviceToHost, e->compute));
-        CK(cudaGetLastError());
-        CK(cudaEventRecord(e->q_end, e->compute));
-        sync_compute(e);
-    };
-    emit();
-    if (tiefix && sm->tie) {
+    const unsigned int err = sm->err;
+    if (err & kErrDupOrders) raise(H2TAP_EDUPKEY, "Q18: duplicate orders primary key (w, d, o_id)");
+    if (err & kErrDupCustomer) raise(H2TAP_EDUPKEY, "Q18: duplicate customer primary key (w, d, c_id)");
+    if (err & kErrDomain) raise(H2TAP_EPLAN, "Q18: join key outside the supported domain");
+    const uint64_t nout = sm->nout;
+    if (sm->tie && nout > 1) {
         // a run of > 32 equal 64-bit prefixes, or a bucket larger than shared memory: redo
         // exactly, one stable LSD radix sort per field (r, then e, then a)
-        SortPairs w = sp2;
+        SortPairs w = q.sp;
+        Q18Plan hp;
+        CK(cudaMemcpy(&hp, q.plan_dev, sizeof hp, cudaMemcpyDeviceToHost));
         launch_iota(w.v[0], nout, e->num_sms, e->compute);
-        const int fb[3] = {sp.bits_r, sp.bits_e, sp.bits_a};
+        const int fb[3] = {hp.spec.bits_r, hp.spec.bits_e, hp.spec.bits_a};
         for (int f = 0; f < 3; ++f) {
-            launch_q18_field_keys(rows, amt, w.v[0], nout, f, sp, w.k[0], e->num_sms, e->compute);
+            launch_q18_field_keys(q.rows, q.amt, w.v[0], nout, f, q.plan_dev, w.k[0], e->num_sms, e->compute);
             const int cur = radix_sort_pairs(nout, fb[f], w, e->num_sms, e->compute);
             if (cur) { std::swap(w.k[0], w.k[1]); std::swap(w.v[0], w.v[1]); }
         }
-        perm = w.v[0];
-        perm_keys = nullptr;  // field keys, not the prefix: amounts are read from amt[]
-        tiefix = false;
-        emit();
+        // keys are field keys, not the prefix: amounts are read from amt[]
+        launch_q18_permute(q.rows, q.amt, w.v[0], nullptr, q.plan_dev, nout, q.out, e->num_sms, e->compute);
+        CK(cudaGetLastError());
     }
-    const Q18Cols &out = r->on_device ? dst : host_dst;
-    add_col(r, "c_last", H2TAP_I32, out.c_last);
-    add_col(r, "c_id", H2TAP_I32, out.c_id);
-    add_col(r, "o_id", H2TAP_I32, out.o_id);
-    add_col(r, "o_entry_d", H2TAP_I64, out.o_entry_d);
-    add_col(r, "o_ol_cnt", H2TAP_I32, out.o_ol_cnt);
-    add_col(r, "amount_sum", H2TAP_I64, out.amount_sum);
-    add_col(r, "o_w_id", H2TAP_I32, out.o_w_id);
-    add_col(r, "o_d_id", H2TAP_I32, out.o_d_id);
+    r->nrows = nout;
+    const void *src[8] = {q.out.c_last, q.out.c_id, q.out.o_id, q.out.o_entry_d, q.out.o_ol_cnt,
+                          q.out.amount_sum, q.out.o_w_id, q.out.o_d_id};
+    const size_t es[8] = {4, 4, 4, 8, 4, 8, 4, 4};
+    if (r->on_device) {
+        for (int i = 0; i < 8; ++i) add_col(r, names[i], types[i], src[i]);
+        give_blocks_to_result(q);
+        if (sm->tie) sync_compute(e);
+        return;
+    }
+    for (int i = 0; i < 8; ++i) {
+        void *h = result_block(r, nout * es[i]);
+        if (nout) CK(cudaMemcpyAsync(h, src[i], nout * es[i], cudaMemcpyDeviceToHost, e->compute));
+        add_col(r, names[i], types[i], h);
+    }
+    sync_compute(e);
+    release_dev_blocks(e, q);
 }
 
 // CH-benCHmark constants as int64 µs UTC / cents (R4, R6).
@@ -958,23 +974,32 @@ constexpr int64_t kQ6DLo = 915148800000000LL;       // 1999-01-01 00:00:00
 constexpr int64_t kQ6DHi = 1577836800000000LL;      // 2020-01-01 00:00:00
 constexpr int64_t kQ18Having = 20000;               // 200.00
 
-h2tap_status query_impl(h2tap_engine *e, uint32_t plan, const int64_t *params, uint32_t nparams,
-                        uint32_t flags, h2tap_result **out) {
-    const auto t0 = std::chrono::steady_clock::now();
-    if (!out) return fail(H2TAP_EINVAL, "out is NULL");
-    *out = nullptr;
-    int64_t p[4];
+h2tap_status parse_query(const h2tap_query &in, QueryCtx &q) {
     uint32_t want;
-    switch (plan) {
-        case H2TAP_Q1: want = 1; p[0] = kQ1Cutoff; break;
-        case H2TAP_Q6: want = 4; p[0] = kQ6DLo; p[1] = kQ6DHi; p[2] = 1; p[3] = 100000; break;
-        case H2TAP_Q18: want = 1; p[0] = kQ18Having; break;
-        default: return fail(H2TAP_EINVAL, "unknown plan id %u", plan);
+    switch (in.plan_id) {
+        case H2TAP_Q1: want = 1; q.p[0] = kQ1Cutoff; break;
+        case H2TAP_Q6: want = 4; q.p[0] = kQ6DLo; q.p[1] = kQ6DHi; q.p[2] = 1; q.p[3] = 100000; break;
+        case H2TAP_Q18: want = 1; q.p[0] = kQ18Having; break;
+        default: return fail(H2TAP_EINVAL, "unknown plan id %u", in.plan_id);
     }
-    if (nparams) {
-        if (nparams != want || !params)
-            return fail(H2TAP_EINVAL, "plan %u takes %u params, got %u", plan, want, nparams);
-        std::memcpy(p, params, sizeof(int64_t) * want);
+    if (in.nparams) {
+        if (in.nparams != want || !in.params)
+            return fail(H2TAP_EINVAL, "plan %u takes %u params, got %u", in.plan_id, want, in.nparams);
+        std::memcpy(q.p, in.params, sizeof(int64_t) * want);
+    }
+    q.plan = in.plan_id;
+    q.flags = in.flags;
+    return H2TAP_OK;
+}
+
+h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2tap_result **out) {
+    const auto t0 = std::chrono::steady_clock::now();
+    if (!out || (n && !qs)) return fail(H2TAP_EINVAL, "queries/out is NULL");
+    for (uint32_t i = 0; i < n; ++i) out[i] = nullptr;
+    std::vector<QueryCtx> ctx(n);
+    for (uint32_t i = 0; i < n; ++i) {
+        const h2tap_status st = parse_query(qs[i], ctx[i]);
+        if (st != H2TAP_OK) return st;
     }
     std::lock_guard<std::mutex> g(e->query_mu);
     CK(cudaSetDevice(e->device));
@@ -985,32 +1010,92 @@ h2tap_status query_impl(h2tap_engine *e, uint32_t plan, const int64_t *params, u
         v = e->published;
     }
     if (!v) return fail(H2TAP_EPLAN, "no snapshot has been published yet");
-    std::unique_ptr<ResultImpl> r(new_result(e, *v, flags & H2TAP_RESULT_DEVICE));
-    e->prof.reset(flags & H2TAP_QUERY_PROFILE, e->compute);
-    // with per-kernel profiling, a short gate lets the whole query be enqueued before the GPU
+    bool profile = false;
+    for (auto &q : ctx) profile |= (q.flags & H2TAP_QUERY_PROFILE) != 0;
+    e->prof.reset(profile, e->compute);
+    // with per-kernel profiling, a short gate lets the whole batch be enqueued before the GPU
     // starts it, so no kernel's event window contains host launch latency
-    if (flags & H2TAP_QUERY_PROFILE) launch_gate(30000, e->compute);
-    const uint64_t launches0 = launches_total();
-    CK(cudaEventRecord(e->q_begin, e->compute));
-    switch (plan) {
-        case H2TAP_Q1: run_q1(e, *v, p, r.get()); break;
-        case H2TAP_Q6: run_q6(e, *v, p, r.get()); break;
-        case H2TAP_Q18: run_q18(e, *v, p, flags, r.get()); break;
+    if (profile) launch_gate(30000, e->compute);
+    struct Cleanup {  // return pooled blocks of queries that did not complete
+        h2tap_engine *e; std::vector<QueryCtx> &c;
+        ~Cleanup() {
+            bool pending = false;
+            for (auto &q : c) pending |= !q.dev_blocks.empty() || q.small.first;
+            if (pending) cudaStreamSynchronize(e->compute);  // kernels may still use the blocks
+            for (auto &q : c) {
+                release_dev_blocks(e, q);
+                if (q.small.first) e->host_pool->put(q.small.first, q.small.second);
+            }
+        }
+    } cleanup{e, ctx};
+    // launch phase: a plan's scratch is reused by a later query of the same plan, so a repeated
+    // plan first completes the queries launched before it
+    size_t done = 0;
+    auto finish_upto = [&](size_t upto) {
+        if (done >= upto) return;
+        sync_compute(e);
+        for (; done < upto; ++done) {
+            QueryCtx &q = ctx[done];
+            switch (q.plan) {
+                case H2TAP_Q1: finish_q1(e, q); break;
+                case H2TAP_Q6: finish_q6(e, q); break;
+                case H2TAP_Q18: finish_q18(e, q); break;
+            }
+        }
+    };
+    for (size_t i = 0; i < ctx.size(); ++i) {
+        QueryCtx &q = ctx[i];
+        for (size_t j = done; j < i; ++j)
+            if (ctx[j].plan == q.plan) { finish_upto(i); break; }
+        q.r.reset(new_result(e, *v, q.flags & H2TAP_RESULT_DEVICE));
+        q.small = e->host_pool->get(256);
+        if (!q.begin) {
+            q.begin = e->prof.ev();
+            q.end = e->prof.ev();
+        }
+        q.mark0 = e->prof.marks.size();
+        q.launches0 = launches_total();
+        CK(cudaEventRecord(q.begin, e->compute));
+        switch (q.plan) {
+            case H2TAP_Q1: launch_q1_plan(e, *v, q); break;
+            case H2TAP_Q6: launch_q6_plan(e, *v, q); break;
+            case H2TAP_Q18: launch_q18_plan(e, *v, q); break;
+        }
+        CK(cudaEventRecord(q.end, e->compute));
+        q.launches = launches_total() - q.launches0;
+        q.mark1 = e->prof.marks.size();
     }
-    float ms = 0;
-    CK(cudaEventElapsedTime(&ms, e->q_begin, e->q_end));
-    r->device_ms = ms;
-    r->kernel_launches = launches_total() - launches0;
-    for (auto &m : e->prof.marks) {
-        float k = 0;
-        CK(cudaEventElapsedTime(&k, m.second.first, m.second.second));
-        r->kname_store.push_back(m.first);
-        r->kms.push_back(k);
+    finish_upto(ctx.size());
+    const double wall = std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - t0).count();
+    for (uint32_t i = 0; i < n; ++i) {
+        QueryCtx &q = ctx[i];
+        ResultImpl *r = q.r.get();
+        float ms = 0;
+        CK(cudaEventElapsedTime(&ms, q.begin, q.end));
+        r->device_ms = ms;
+        r->kernel_launches = q.launches;
+        for (size_t m = q.mark0; m < q.mark1; ++m) {
+            float k = 0;
+            CK(cudaEventElapsedTime(&k, e->prof.marks[m].second.first, e->prof.marks[m].second.second));
+            r->kname_store.push_back(e->prof.marks[m].first);
+            r->kms.push_back(k);
+        }
+        r->e2e_ms = wall;
+        e->host_pool->put(q.small.first, q.small.second);
+        q.small = {};
     }
-    r->e2e_ms = std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - t0).count();
-    r->finish();
-    *out = r.release();
+    for (uint32_t i = 0; i < n; ++i) {
+        ctx[i].r->finish();
+        out[i] = ctx[i].r.release();
+    }
     return H2TAP_OK;
+}
+
+h2tap_status query_impl(h2tap_engine *e, uint32_t plan, const int64_t *params, uint32_t nparams,
+                        uint32_t flags, h2tap_result **out) {
+    if (!out) return fail(H2TAP_EINVAL, "out is NULL");
+    h2tap_query q{plan, nparams, params, flags};
+    return queries_impl(e, &q, 1, out);
 }
 
 template <class F> h2tap_status guarded(F &&f) {
@@ -1103,6 +1188,12 @@ h2tap_status h2tap_run_query_ex(h2tap_engine *e, uint32_t plan_id, const int64_t
 h2tap_status h2tap_run_query(h2tap_engine *e, uint32_t plan_id, const int64_t *params,
                              uint32_t nparams, h2tap_result **out) {
     return h2tap_run_query_ex(e, plan_id, params, nparams, 0, out);
+}
+
+h2tap_status h2tap_run_queries(h2tap_engine *e, const h2tap_query *queries, uint32_t nqueries,
+                               h2tap_result **out) {
+    if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
+    return guarded([&] { return queries_impl(e, queries, nqueries, out); });
 }
 
 void h2tap_free(h2tap_result *r) {

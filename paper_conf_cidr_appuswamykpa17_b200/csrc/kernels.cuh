@@ -45,7 +45,8 @@ void launch_q1(const int32_t *number, const int64_t *deliv, const int32_t *qty,
                cudaStream_t st);
 void launch_q1_compact(const Q1Scratch &s, cudaStream_t st);        // tables -> groups[], ngroups
 void launch_q1_merge(const Q1Group *all, uint64_t n, const Q1Scratch &s, cudaStream_t st);
-void launch_q1_emit(const Q1Scratch &s, uint64_t ngroups, cudaStream_t st);  // rank by key + AVG
+void launch_q1_emit(const Q1Scratch &s, uint64_t max_groups, cudaStream_t st);  // rank by key + AVG;
+                                                                           // reads *ngroups on device
 
 // ------------------------------------------------------------ Q18 (K3-K5) --
 struct HtSlot { unsigned long long key; unsigned int row; unsigned int pad; };  // 16 B
@@ -134,9 +135,12 @@ struct BucketSort {
     unsigned int *offset;  // [2^kBucketMaxBits + 1]
     unsigned int *big;     // [1 + 2^kBucketMaxBits]: count, then ids of buckets > small capacity
 };
-// Sorted pairs end in k[1]/v[1] (input in k[0]/v[0]).
-void bucket_sort_pairs(uint64_t n, int bits, int bucket_bits, const BucketSort &s, unsigned int *flag,
-                       int num_sms, cudaStream_t st);
+// Sorted pairs end in k[1]/v[1] (input in k[0]/v[0]). The row count and the bucket shift are
+// read on the device (*dn, *dshift), so the whole ORDER BY runs without a host round trip;
+// `n_max` (an upper bound of *dn) only sizes the grids.
+void bucket_sort_pairs(uint64_t n_max, const unsigned long long *dn, const int *dshift,
+                       int bucket_bits, const BucketSort &s, unsigned int *flag, int num_sms,
+                       cudaStream_t st);
 
 // Q18 ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id (R11).
 struct Q18SortSpec {         // host-computed from Q18Stats
@@ -146,21 +150,33 @@ struct Q18SortSpec {         // host-computed from Q18Stats
     int bits_a, bits_e, bits_r;  // field widths: amount (desc), entry, row rank
     int prefix_bits;         // width of the sorted 64-bit prefix of the composite key
 };
-void launch_q18_sort_keys(const Q18Row *rows, const long long *amt, uint64_t n,
-                          const Q18SortSpec &spec, const SortPairs &s, int num_sms, cudaStream_t st);
+// Device-side plan of the ORDER BY, computed from the HAVING kernel's statistics and row count
+// (no host round trip): field widths, 64-bit prefix width, whether a tie-fix is needed, and the
+// bucket shift for `bucket_bits` buckets.
+struct Q18Plan {
+    unsigned long long n;
+    Q18SortSpec spec;
+    int tiefix;
+    int shift;
+};
+void launch_q18_plan(const Q18Stats *stats, const unsigned long long *nout, int bucket_bits,
+                     Q18Plan *plan, cudaStream_t st);
+void launch_q18_sort_keys(const Q18Row *rows, const long long *amt, const Q18Plan *plan,
+                          uint64_t n_max, const SortPairs &s, int num_sms, cudaStream_t st);
 // Within runs of equal prefix, order by the full tuple; runs longer than 32 raise *flag.
 void launch_q18_tiefix(const Q18Row *rows, const long long *amt, const unsigned long long *keys,
-                       unsigned int *vals, uint64_t n, unsigned int *flag, int num_sms,
-                       cudaStream_t st);
+                       unsigned int *vals, const Q18Plan *plan, uint64_t n_max, unsigned int *flag,
+                       int num_sms, cudaStream_t st);
 // Exact fallback: three stable passes over the full fields (row rank, entry, amount).
 void launch_q18_field_keys(const Q18Row *rows, const long long *amt, const unsigned int *vals,
-                           uint64_t n, int field, const Q18SortSpec &spec, unsigned long long *keys,
+                           uint64_t n, int field, const Q18Plan *plan, unsigned long long *keys,
                            int num_sms, cudaStream_t st);
 void launch_iota(unsigned int *v, uint64_t n, int num_sms, cudaStream_t st);
 // Gather rows in `perm` order into SoA columns. amount_sum: decoded from the sorted prefix keys
 // when `keys` is given (field a is always whole at the top of the prefix), else read from amt.
+// `perm`/`keys` null: identity order (n <= 1) or amounts read from amt (field-key fallback).
 void launch_q18_permute(const Q18Row *rows, const long long *amt, const unsigned int *perm,
-                        const unsigned long long *keys, const Q18SortSpec &spec, uint64_t n,
+                        const unsigned long long *keys, const Q18Plan *plan, uint64_t n_max,
                         const Q18Cols &dst, int num_sms, cudaStream_t st);
 
 // ------------------------------------------------------------ store (a1) --

@@ -362,8 +362,10 @@ __global__ void q1_merge_kernel(const Q1Group *__restrict__ all, uint64_t n, Q1S
 
 // ORDER BY ol_number: keys are distinct, so each group's output position is its rank
 // (number of smaller keys). AVG = SUM / COUNT in IEEE double, money / 100 (R7).
-__global__ void q1_emit_kernel(Q1Scratch g, uint64_t ng) {
+__global__ void q1_emit_kernel(Q1Scratch g) {
     __shared__ long long tile[1024];
+    const uint64_t ng = *g.ngroups;  // read on the device: no host round trip before emitting
+    if ((uint64_t)blockIdx.x * blockDim.x >= ng) return;  // grid sized for the maximum
     const uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
     const long long mine = i < ng ? g.groups[i].key : 0;
     uint64_t rank = 0;
@@ -444,9 +446,8 @@ void launch_q1_merge(const Q1Group *all, uint64_t n, const Q1Scratch &s, cudaStr
     count_launches(1);
 }
 
-void launch_q1_emit(const Q1Scratch &s, uint64_t ngroups, cudaStream_t st) {
-    if (!ngroups) return;
-    q1_emit_kernel<<<(unsigned)((ngroups + 255) / 256), 256, 0, st>>>(s, ngroups);
+void launch_q1_emit(const Q1Scratch &s, uint64_t max_groups, cudaStream_t st) {
+    q1_emit_kernel<<<(unsigned)((max_groups + 255) / 256), 256, 0, st>>>(s);
     count_launches(1);
 }
 

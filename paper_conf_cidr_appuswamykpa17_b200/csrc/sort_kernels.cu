@@ -186,8 +186,10 @@ __device__ __forceinline__ unsigned long long prefix_key(const Q18Row &r, long l
 }
 
 __global__ void sort_keys_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
-                                 uint64_t n, Q18SortSpec sp, unsigned long long *__restrict__ k,
+                                 const Q18Plan *__restrict__ plan, unsigned long long *__restrict__ k,
                                  unsigned int *__restrict__ v) {
+    const uint64_t n = plan->n;
+    const Q18SortSpec sp = plan->spec;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
         k[i] = prefix_key(rows[i], amt[i], sp);
@@ -208,7 +210,9 @@ constexpr int kMaxRun = 32;
 
 __global__ void tiefix_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
                               const unsigned long long *__restrict__ k, unsigned int *__restrict__ v,
-                              uint64_t n, unsigned int *flag) {
+                              const Q18Plan *__restrict__ plan, unsigned int *flag) {
+    if (!plan->tiefix) return;  // composite key fits 64 bits: keys are distinct
+    const uint64_t n = plan->n;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
         const unsigned long long ki = k[i];
@@ -234,7 +238,8 @@ __global__ void tiefix_kernel(const Q18Row *__restrict__ rows, const long long *
 
 __global__ void field_keys_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
                                   const unsigned int *__restrict__ vals, uint64_t n, int field,
-                                  Q18SortSpec sp, unsigned long long *__restrict__ k) {
+                                  const Q18Plan *__restrict__ plan, unsigned long long *__restrict__ k) {
+    const Q18SortSpec sp = plan->spec;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
         const unsigned int x = vals[i];
@@ -253,8 +258,11 @@ __global__ void iota_kernel(unsigned int *v, uint64_t n) {
 // amount_sum comes from the sorted prefix key (contiguous) instead of a second random gather.
 __global__ void permute_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
                                const unsigned int *__restrict__ perm,
-                               const unsigned long long *__restrict__ keys, Q18SortSpec sp,
-                               uint64_t n, Q18Cols dst) {
+                               const unsigned long long *__restrict__ keys,
+                               const Q18Plan *__restrict__ plan, Q18Cols dst) {
+    const uint64_t n = plan->n;
+    const Q18SortSpec sp = plan->spec;
+    if (n <= 1) { perm = nullptr; keys = nullptr; }  // nothing was sorted
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     const int ashift = sp.prefix_bits - sp.bits_a;
     for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < n; j += stride) {
@@ -278,6 +286,33 @@ __global__ void permute_kernel(const Q18Row *__restrict__ rows, const long long 
     }
 }
 
+__device__ __forceinline__ int bitwidth_dev(unsigned long long x) { return x ? 64 - __clzll(x) : 0; }
+
+// One thread: the ORDER BY plan from the HAVING statistics (widths of a, e, r; prefix width).
+__global__ void q18_plan_kernel(const Q18Stats *__restrict__ stats, const unsigned long long *nout,
+                                int bucket_bits, Q18Plan *plan) {
+    const Q18Stats st = *stats;
+    Q18Plan p{};
+    p.n = *nout;
+    Q18SortSpec &sp = p.spec;
+    if (p.n > 1) {
+        sp.amt_max = st.amt_max;
+        sp.ent_min = st.ent_min;
+        sp.w_min = st.w_min; sp.d_min = st.d_min; sp.o_min = st.o_min;
+        sp.nd = (long long)st.d_max - st.d_min + 1;
+        sp.no = (long long)st.o_max - st.o_min + 1;
+        const unsigned long long nw = (unsigned long long)((long long)st.w_max - st.w_min + 1);
+        sp.bits_a = bitwidth_dev((unsigned long long)st.amt_max - (unsigned long long)st.amt_min);
+        sp.bits_e = bitwidth_dev((unsigned long long)st.ent_max - (unsigned long long)st.ent_min);
+        sp.bits_r = bitwidth_dev(nw * (unsigned long long)sp.nd * (unsigned long long)sp.no - 1);
+        const int B = sp.bits_a + sp.bits_e + sp.bits_r;
+        sp.prefix_bits = B <= 64 ? B : 64;
+        p.tiefix = B > 64;
+        p.shift = sp.prefix_bits > bucket_bits ? sp.prefix_bits - bucket_bits : 0;
+    }
+    *plan = p;
+}
+
 unsigned grid_cap(uint64_t work, int threads, int num_sms, int per_sm) {
     uint64_t want = (work + threads - 1) / threads;
     uint64_t cap = (uint64_t)num_sms * per_sm;
@@ -286,6 +321,12 @@ unsigned grid_cap(uint64_t work, int threads, int num_sms, int per_sm) {
 }
 
 }  // namespace
+
+void launch_q18_plan(const Q18Stats *stats, const unsigned long long *nout, int bucket_bits,
+                     Q18Plan *plan, cudaStream_t st) {
+    q18_plan_kernel<<<1, 1, 0, st>>>(stats, nout, bucket_bits, plan);
+    count_launches(1);
+}
 
 int radix_sort_pairs(uint64_t n, int bits, const SortPairs &s, int num_sms, cudaStream_t st) {
     (void)num_sms;
@@ -304,23 +345,23 @@ int radix_sort_pairs(uint64_t n, int bits, const SortPairs &s, int num_sms, cuda
     return cur;
 }
 
-void launch_q18_sort_keys(const Q18Row *rows, const long long *amt, uint64_t n,
-                          const Q18SortSpec &spec, const SortPairs &s, int num_sms, cudaStream_t st) {
-    sort_keys_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, amt, n, spec, s.k[0], s.v[0]);
+void launch_q18_sort_keys(const Q18Row *rows, const long long *amt, const Q18Plan *plan,
+                          uint64_t n_max, const SortPairs &s, int num_sms, cudaStream_t st) {
+    sort_keys_kernel<<<grid_cap(n_max, 256, num_sms, 8), 256, 0, st>>>(rows, amt, plan, s.k[0], s.v[0]);
     count_launches(1);
 }
 
 void launch_q18_tiefix(const Q18Row *rows, const long long *amt, const unsigned long long *keys,
-                       unsigned int *vals, uint64_t n, unsigned int *flag, int num_sms,
-                       cudaStream_t st) {
-    tiefix_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, amt, keys, vals, n, flag);
+                       unsigned int *vals, const Q18Plan *plan, uint64_t n_max, unsigned int *flag,
+                       int num_sms, cudaStream_t st) {
+    tiefix_kernel<<<grid_cap(n_max, 256, num_sms, 8), 256, 0, st>>>(rows, amt, keys, vals, plan, flag);
     count_launches(1);
 }
 
 void launch_q18_field_keys(const Q18Row *rows, const long long *amt, const unsigned int *vals,
-                           uint64_t n, int field, const Q18SortSpec &spec, unsigned long long *keys,
+                           uint64_t n, int field, const Q18Plan *plan, unsigned long long *keys,
                            int num_sms, cudaStream_t st) {
-    field_keys_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, amt, vals, n, field, spec, keys);
+    field_keys_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, amt, vals, n, field, plan, keys);
     count_launches(1);
 }
 
@@ -330,9 +371,9 @@ void launch_iota(unsigned int *v, uint64_t n, int num_sms, cudaStream_t st) {
 }
 
 void launch_q18_permute(const Q18Row *rows, const long long *amt, const unsigned int *perm,
-                        const unsigned long long *keys, const Q18SortSpec &spec, uint64_t n,
+                        const unsigned long long *keys, const Q18Plan *plan, uint64_t n_max,
                         const Q18Cols &dst, int num_sms, cudaStream_t st) {
-    permute_kernel<<<grid_cap(n, 256, num_sms, 8), 256, 0, st>>>(rows, amt, perm, keys, spec, n, dst);
+    permute_kernel<<<grid_cap(n_max, 256, num_sms, 8), 256, 0, st>>>(rows, amt, perm, keys, plan, dst);
     count_launches(1);
 }
 
@@ -355,8 +396,10 @@ constexpr int kLsCapLarge = 8192;                  // rows per bucket: large-buc
 constexpr int kLsSubMax = 1024;                    // max sub-buckets per bucket
 
 __global__ void __launch_bounds__(kBkThreads)
-bucket_hist_kernel(const unsigned long long *__restrict__ key, uint64_t n, int shift, int nb,
-                   unsigned int *__restrict__ count) {
+bucket_hist_kernel(const unsigned long long *__restrict__ key, const unsigned long long *dn,
+                   const int *dshift, int nb, unsigned int *__restrict__ count) {
+    const uint64_t n = *dn;
+    const int shift = *dshift;
     extern __shared__ unsigned int h[];
     for (int i = threadIdx.x; i < nb; i += kBkThreads) h[i] = 0;
     __syncthreads();
@@ -427,8 +470,12 @@ __global__ void __launch_bounds__(1024) bucket_scan_kernel(unsigned int *__restr
 // scatter into buckets: a block's shared histogram reserves one global range per bucket
 __global__ void __launch_bounds__(kBkThreads)
 bucket_scatter_kernel(const unsigned long long *__restrict__ kin, const unsigned int *__restrict__ vin,
-                      unsigned long long *__restrict__ kout, unsigned int *__restrict__ vout, uint64_t n,
-                      int shift, int nb, unsigned int *__restrict__ cursor) {
+                      unsigned long long *__restrict__ kout, unsigned int *__restrict__ vout,
+                      const unsigned long long *dn, const int *dshift, int nb,
+                      unsigned int *__restrict__ cursor) {
+    const uint64_t n = *dn;
+    const int shift = *dshift;
+    if ((uint64_t)blockIdx.x * kBkThreads * kBkItems >= n) return;  // grid sized for an upper bound
     extern __shared__ unsigned int h[];  // [nb] local counts -> local cursors
     for (int i = threadIdx.x; i < nb; i += kBkThreads) h[i] = 0;
     const uint64_t base = (uint64_t)blockIdx.x * kBkThreads * kBkItems;
@@ -476,8 +523,9 @@ template <int kLsCap> struct LsSmem {
 template <int kLsCap, int kMin>
 __global__ void __launch_bounds__(kBkThreads)
 bucket_local_sort_kernel(unsigned long long *__restrict__ k, unsigned int *__restrict__ v,
-                         const unsigned int *__restrict__ offset, int nb, int shift,
+                         const unsigned int *__restrict__ offset, int nb, const int *dshift,
                          unsigned int *flag, unsigned int *big) {
+    const int shift = *dshift;
     extern __shared__ __align__(16) unsigned char smem_raw[];
     LsSmem<kLsCap> &S = *reinterpret_cast<LsSmem<kLsCap> *>(smem_raw);
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -564,12 +612,11 @@ bucket_local_sort_kernel(unsigned long long *__restrict__ k, unsigned int *__res
 
 }  // namespace
 
-void bucket_sort_pairs(uint64_t n, int bits, int bucket_bits, const BucketSort &s, unsigned int *flag,
-                       int num_sms, cudaStream_t st) {
-    if (bucket_bits > bits) bucket_bits = bits;
+void bucket_sort_pairs(uint64_t n_max, const unsigned long long *dn, const int *dshift,
+                       int bucket_bits, const BucketSort &s, unsigned int *flag, int num_sms,
+                       cudaStream_t st) {
     if (bucket_bits > kBucketMaxBits) bucket_bits = kBucketMaxBits;
     const int nb = 1 << bucket_bits;
-    const int shift = bits - bucket_bits;
     static bool init = false;
     if (!init) {
         cudaFuncSetAttribute(bucket_local_sort_kernel<kLsCapSmall, 0>,
@@ -585,25 +632,25 @@ void bucket_sort_pairs(uint64_t n, int bits, int bucket_bits, const BucketSort &
     cudaMemsetAsync(s.count, 0, sizeof(unsigned int) * (nb + 1), st);
     cudaMemsetAsync(s.big, 0, sizeof(unsigned int), st);
     const uint64_t per = (uint64_t)kBkThreads * kBkItems;
-    uint64_t hb = (n + per - 1) / per;
+    uint64_t hb = (n_max + per - 1) / per;
     if (hb > (uint64_t)num_sms * 2) hb = (uint64_t)num_sms * 2;
     if (!hb) hb = 1;
-    bucket_hist_kernel<<<(unsigned)hb, kBkThreads, nb * 4, st>>>(s.k[0], n, shift, nb, s.count);
+    bucket_hist_kernel<<<(unsigned)hb, kBkThreads, nb * 4, st>>>(s.k[0], dn, dshift, nb, s.count);
     count_launches(1);
     bucket_scan_kernel<<<1, 1024, 0, st>>>(s.count, nb, s.offset, s.cursor);
     count_launches(1);
-    const uint64_t sb = (n + per - 1) / per;
+    const uint64_t sb = (n_max + per - 1) / per;
     bucket_scatter_kernel<<<(unsigned)(sb ? sb : 1), kBkThreads, nb * 4, st>>>(
-        s.k[0], s.v[0], s.k[1], s.v[1], n, shift, nb, s.cursor);
+        s.k[0], s.v[0], s.k[1], s.v[1], dn, dshift, nb, s.cursor);
     count_launches(1);
     unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
     bucket_local_sort_kernel<kLsCapSmall, 0><<<lb, kBkThreads, sizeof(LsSmem<kLsCapSmall>), st>>>(
-        s.k[1], s.v[1], s.offset, nb, shift, flag, s.big);
+        s.k[1], s.v[1], s.offset, nb, dshift, flag, s.big);
     count_launches(1);
     // buckets above the small capacity (skewed keys): one block per SM, ~200 KB shared memory
     bucket_local_sort_kernel<kLsCapLarge, kLsCapSmall><<<(unsigned)num_sms, kBkThreads,
                                                           sizeof(LsSmem<kLsCapLarge>), st>>>(
-        s.k[1], s.v[1], s.offset, nb, shift, flag, s.big);
+        s.k[1], s.v[1], s.offset, nb, dshift, flag, s.big);
     count_launches(1);
 }
 

@@ -278,6 +278,34 @@ def test_profile_reports_kernels(h, eng, L):
     r.free()
 
 
+def test_batch_queries_one_epoch(h, eng, L):
+    """h2tap_run_queries: several plans (repeats included) enqueued back to back, one sync."""
+    t = chgen.generate(1, 3, seed=27)
+    L.load(t)
+    batch = [(6, None, 0), (1, None, h.H2TAP_RESULT_DEVICE), (18, [Q18_HAVING], 0),
+             (18, [5_000_000], h.H2TAP_RESULT_DEVICE | HASH), (6, [Q6_D_LO, Q6_D_HI, 3, 7], 0),
+             (1, [chgen.TS_1995], h.H2TAP_QUERY_PROFILE)]
+    rs = h.h2tap_run_queries(eng, batch)
+    try:
+        got = []
+        for r in rs:
+            x = r.to_numpy()
+            x["_nulls"] = dict(r.nulls)
+            got.append(x)
+        assert len({r.epoch for r in rs}) == 1
+    finally:
+        for r in rs:
+            r.free()
+    assert_q6(got[0], oracle.q6(t, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))
+    assert_q1(got[1], oracle.q1(t, Q1_CUTOFF))
+    assert_q18(got[2], oracle.q18(t, Q18_HAVING))
+    assert_q18(got[3], oracle.q18(t, 5_000_000))
+    assert_q6(got[4], oracle.q6(t, Q6_D_LO, Q6_D_HI, 3, 7))
+    assert_q1(got[5], oracle.q1(t, chgen.TS_1995))
+    with pytest.raises(h.H2tapError):
+        h.h2tap_run_queries(eng, [(6, None, 0), (99, None, 0)])
+
+
 # ------------------------------------------------------- snapshot semantics --
 def test_snapshot_epochs_append_and_errors(h):
     """a1: append-only refresh, epoch monotonicity, shape errors, async publish."""
