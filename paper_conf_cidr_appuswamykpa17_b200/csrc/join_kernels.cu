@@ -14,6 +14,7 @@
 #include <cstdint>
 #include <cuda_runtime.h>
 
+#include "cache_hints.cuh"
 #include "kernels.cuh"
 
 namespace h2tap {
@@ -330,6 +331,7 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
     __shared__ unsigned int wsum[kHavingThreads / 32];
     __shared__ unsigned long long s_base;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const uint64_t keep = l2_policy_evict_last();
     StatAcc stat;
     for (uint64_t base = (uint64_t)blockIdx.x * kHavingRows; base < n;
          base += (uint64_t)gridDim.x * kHavingRows) {
@@ -394,7 +396,11 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
         for (int u = 0; u < kHavingUnroll; ++u) {
             if (crow[u] == kNoRow) continue;
             s.amt[p] = sum[u];
-            s.rows[p++] = row[u];
+            // result rows are gathered again by the ORDER BY permute: keep them in L2
+            const unsigned long long *w64 = reinterpret_cast<const unsigned long long *>(&row[u]);
+            st16_policy(s.rows + p, w64[0], w64[1], keep);
+            st16_policy(reinterpret_cast<char *>(s.rows + p) + 16, w64[2], w64[3], keep);
+            ++p;
             stat.add(sum[u], row[u].o_entry_d, w[u], d[u], row[u].o_id);
         }
         __syncthreads();  // wsum / s_base reuse

@@ -248,8 +248,28 @@ q1_kernel(const int4 *__restrict__ number, const longlong2 *__restrict__ deliv,
     const uint64_t nvec = n >> 2;
     const uint64_t gwarp = ((uint64_t)blockIdx.x * kQ1Threads + tid) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * kQ1Threads) >> 5;
-    // warp-uniform trip count so that ballots in the sparse path are convergent
-    for (uint64_t base = gwarp * 32 * kQ1Unroll; base < nvec; base += nwarps * 32 * kQ1Unroll) {
+    // warp-uniform trip count so that ballots in the sparse path are convergent. Software
+    // pipeline: the next iteration's 12 loads are issued before this iteration's rows are
+    // aggregated, so HBM requests stay in flight during the shared-memory updates.
+    const uint64_t step = nwarps * 32 * kQ1Unroll;
+    int4 pnb[kQ1Unroll], pqv[kQ1Unroll];
+    longlong2 pd0[kQ1Unroll], pd1[kQ1Unroll], pa0[kQ1Unroll], pa1[kQ1Unroll];
+    auto load = [&](uint64_t base) {
+#pragma unroll
+        for (int u = 0; u < kQ1Unroll; ++u) {
+            const uint64_t x = base + u * 32 + lane;
+            if (x < nvec) {
+                pnb[u] = ld_stream(number + x);
+                pd0[u] = ld_stream(deliv + 2 * x);
+                pd1[u] = ld_stream(deliv + 2 * x + 1);
+                pqv[u] = ld_stream(qty + x);
+                pa0[u] = ld_stream(amt + 2 * x);
+                pa1[u] = ld_stream(amt + 2 * x + 1);
+            }
+        }
+    };
+    load(gwarp * 32 * kQ1Unroll);
+    for (uint64_t base = gwarp * 32 * kQ1Unroll; base < nvec; base += step) {
         int4 nb[kQ1Unroll], qv[kQ1Unroll];
         longlong2 d0[kQ1Unroll], d1[kQ1Unroll], a0[kQ1Unroll], a1[kQ1Unroll];
         bool ok[kQ1Unroll];
@@ -258,18 +278,14 @@ q1_kernel(const int4 *__restrict__ number, const longlong2 *__restrict__ deliv,
             const uint64_t x = base + u * 32 + lane;
             ok[u] = x < nvec;
             if (ok[u]) {
-                nb[u] = ld_stream(number + x);
-                d0[u] = ld_stream(deliv + 2 * x);
-                d1[u] = ld_stream(deliv + 2 * x + 1);
-                qv[u] = ld_stream(qty + x);
-                a0[u] = ld_stream(amt + 2 * x);
-                a1[u] = ld_stream(amt + 2 * x + 1);
+                nb[u] = pnb[u]; d0[u] = pd0[u]; d1[u] = pd1[u]; qv[u] = pqv[u]; a0[u] = pa0[u]; a1[u] = pa1[u];
             } else {
                 nb[u] = make_int4(0, 0, 0, 0); qv[u] = nb[u];
                 d0[u] = make_longlong2(kNullTs, kNullTs); d1[u] = d0[u];
                 a0[u] = make_longlong2(0, 0); a1[u] = a0[u];
             }
         }
+        load(base + step);
         bool sp[kQ1Unroll][4];
 #pragma unroll
         for (int u = 0; u < kQ1Unroll; ++u) {

@@ -14,6 +14,7 @@
 #include <cstdint>
 #include <cuda_runtime.h>
 
+#include "cache_hints.cuh"
 #include "kernels.cuh"
 
 namespace h2tap {
@@ -265,9 +266,15 @@ __global__ void permute_kernel(const Q18Row *__restrict__ rows, const long long 
     if (n <= 1) { perm = nullptr; keys = nullptr; }  // nothing was sorted
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     const int ashift = sp.prefix_bits - sp.bits_a;
+    const uint64_t drop = l2_policy_evict_first();  // last read of the result rows
     for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < n; j += stride) {
         const unsigned int i = perm ? perm[j] : (unsigned int)j;
-        const Q18Row r = rows[i];
+        Q18Row r;
+        {
+            unsigned long long *w64 = reinterpret_cast<unsigned long long *>(&r);
+            ld16_policy(rows + i, w64[0], w64[1], drop);
+            ld16_policy(reinterpret_cast<const char *>(rows + i) + 16, w64[2], w64[3], drop);
+        }
         long long amount;
         if (keys) {
             const unsigned long long a = sp.bits_a ? (__ldcs(keys + j) >> ashift) : 0ull;
