@@ -34,7 +34,8 @@ import numpy as np
 __all__ = [
     "Scale", "TINY", "FULL", "NULL_TS", "LOAD_TS", "TS_1995", "TS_2025",
     "DAY_US", "ts_us", "generate", "generate_item", "neworder_delta",
-    "warehouse_ranges", "concat_tables", "TABLE_COLUMNS",
+    "warehouse_ranges", "concat_tables", "TABLE_COLUMNS", "NewOrderState", "neworder_batch",
+    "ROW_DTYPES", "to_records",
 ]
 
 
@@ -258,3 +259,63 @@ def neworder_delta(state: NewOrderState, n_txn: int, *, seed: int, batch: int,
     dts = {c: dt for t in ("orders", "order_line") for c, dt in TABLE_COLUMNS[t]}
     return {"orders": {k: np.asarray(v, dtype=dts[k]) for k, v in cols_o.items()},
             "order_line": {k: np.asarray(v, dtype=dts[k]) for k, v in cols_l.items()}}
+
+
+def neworder_batch(state: NewOrderState, n_txn: int, *, seed: int, batch: int, item=None):
+    """Vectorised ``neworder_delta``: the rows appended by ``n_txn`` NewOrder transactions
+    (district and customer uniform, ol_cnt U[5,15], item uniform, qty U[1,10],
+    amount = qty * i_price, delivery NULL, o_id = next id of the district, o_entry_d a logical
+    clock). Same semantics as ``neworder_delta``; used to drive config C5 at high rates."""
+    sc = state.scale
+    rng = np.random.Generator(np.random.Philox(key=np.array([seed, 1 << 41 | batch], dtype=np.uint64)))
+    if item is None:
+        item = generate_item(seed, sc)
+    w = rng.integers(state.w_lo, state.w_hi, size=n_txn).astype(np.int32)
+    d = rng.integers(1, sc.districts + 1, size=n_txn).astype(np.int32)
+    c = rng.integers(1, sc.customers_per_district + 1, size=n_txn).astype(np.int32)
+    cnt = rng.integers(sc.min_ol_cnt, sc.max_ol_cnt + 1, size=n_txn).astype(np.int32)
+    # o_id: next id per (w, d), in transaction order
+    key = w.astype(np.int64) * 64 + d
+    order = np.argsort(key, kind="stable")
+    ks = key[order]
+    first = np.r_[True, ks[1:] != ks[:-1]]
+    grp_start = np.maximum.accumulate(np.where(first, np.arange(n_txn), 0))
+    rank_in_grp = np.arange(n_txn) - grp_start
+    base = np.array([state.next_o_id.get((int(k) // 64, int(k) % 64), sc.orders_per_district + 1)
+                     for k in ks[first]], dtype=np.int64)
+    gid = np.cumsum(first) - 1
+    o_sorted = base[gid] + rank_in_grp
+    o_id = np.empty(n_txn, np.int64)
+    o_id[order] = o_sorted
+    for k, b, g in zip(ks[first], base, np.bincount(gid)):
+        state.next_o_id[(int(k) // 64, int(k) % 64)] = int(b + g)
+    entry = state.clock + 1_000 * np.arange(1, n_txn + 1, dtype=np.int64)
+    state.clock = int(entry[-1]) if n_txn else state.clock
+    n_ol = int(cnt.sum())
+    starts = np.zeros(n_txn, np.int64)
+    np.cumsum(cnt[:-1], out=starts[1:])
+    number = (np.arange(n_ol) - np.repeat(starts, cnt) + 1).astype(np.int32)
+    iid = rng.integers(1, sc.items + 1, size=n_ol).astype(np.int32)
+    qty = rng.integers(1, 11, size=n_ol).astype(np.int32)
+    amount = qty.astype(np.int64) * item["i_price"][iid - 1]
+    orders = {"o_w_id": w, "o_d_id": d, "o_id": o_id.astype(np.int32), "o_c_id": c, "o_ol_cnt": cnt,
+              "o_carrier_id": np.full(n_txn, -1, np.int32), "o_all_local": np.ones(n_txn, np.int32),
+              "o_entry_d": entry}
+    ol = {"ol_w_id": np.repeat(w, cnt), "ol_d_id": np.repeat(d, cnt),
+          "ol_o_id": np.repeat(o_id.astype(np.int32), cnt), "ol_number": number, "ol_i_id": iid,
+          "ol_supply_w_id": np.repeat(w, cnt), "ol_delivery_d": np.full(n_ol, NULL_TS, np.int64),
+          "ol_quantity": qty, "ol_amount": amount}
+    return {"orders": orders, "order_line": ol}
+
+
+# NSM record layouts of the host row store (one record per row, fields in schema order)
+ROW_DTYPES = {t: np.dtype([(c, dt) for c, dt in cols]) for t, cols in TABLE_COLUMNS.items()}
+
+
+def to_records(table: str, cols: dict) -> np.ndarray:
+    """Columns -> NSM records (numpy structured array) of ``table``'s row layout."""
+    n = len(next(iter(cols.values())))
+    rec = np.empty(n, ROW_DTYPES[table])
+    for c in ROW_DTYPES[table].names:
+        rec[c] = cols[c]
+    return rec

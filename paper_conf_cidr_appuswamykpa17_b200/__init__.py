@@ -67,6 +67,16 @@ class h2tap_table(C.Structure):
                 ("row_count", C.c_uint64), ("first_row", C.c_uint64), ("flags", C.c_uint32)]
 
 
+class h2tap_field(C.Structure):
+    _fields_ = [("column_id", C.c_uint32), ("type", C.c_uint32), ("offset", C.c_uint32)]
+
+
+class h2tap_row_table(C.Structure):
+    _fields_ = [("table_id", C.c_uint32), ("nfields", C.c_uint32), ("fields", C.POINTER(h2tap_field)),
+                ("records", C.c_void_p), ("record_size", C.c_uint64), ("row_count", C.c_uint64),
+                ("first_row", C.c_uint64), ("flags", C.c_uint32)]
+
+
 class h2tap_config(C.Structure):
     _fields_ = [("device", C.c_int), ("rank", C.c_int), ("world", C.c_int),
                 ("nccl_unique_id", C.c_void_p)]
@@ -92,6 +102,9 @@ _lib.h2tap_open.argtypes = [C.POINTER(h2tap_config), C.POINTER(_P)]
 _lib.h2tap_load_snapshot_ex.argtypes = [_P, C.POINTER(h2tap_table), C.c_uint32, C.c_uint64, C.c_uint32]
 _lib.h2tap_load_snapshot.argtypes = [_P, C.POINTER(h2tap_table), C.c_uint32, C.c_uint64]
 _lib.h2tap_sync.argtypes = [_P, C.POINTER(C.c_uint64)]
+_lib.h2tap_reserve.argtypes = [_P, C.c_uint32, C.c_uint64]
+_lib.h2tap_load_snapshot_rows.argtypes = [_P, C.POINTER(h2tap_row_table), C.c_uint32, C.c_uint64,
+                                          C.c_uint32]
 _lib.h2tap_run_query_ex.argtypes = [_P, C.c_uint32, C.POINTER(C.c_int64), C.c_uint32, C.c_uint32,
                                     C.POINTER(C.POINTER(h2tap_result))]
 _lib.h2tap_run_query.argtypes = [_P, C.c_uint32, C.POINTER(C.c_int64), C.c_uint32,
@@ -106,12 +119,15 @@ _lib.h2tap_last_error.restype = C.c_char_p
 _lib.h2tap_nccl_unique_id.argtypes = [_P]
 _lib.h2tap_compute_stream.argtypes = [_P, C.POINTER(_P)]
 _lib.h2tap_c_last_name.argtypes = [C.c_int32, C.c_char_p, C.c_size_t]
-for _f in ("h2tap_open", "h2tap_load_snapshot_ex", "h2tap_load_snapshot", "h2tap_sync",
+for _f in ("h2tap_open", "h2tap_load_snapshot_ex", "h2tap_load_snapshot", "h2tap_load_snapshot_rows",
+           "h2tap_reserve",
+           "h2tap_sync",
            "h2tap_run_query_ex", "h2tap_run_query", "h2tap_run_queries", "h2tap_nccl_unique_id",
            "h2tap_compute_stream"):
     getattr(_lib, _f).restype = C.c_int
 
-ABI_SYMBOLS = ["h2tap_open", "h2tap_load_snapshot", "h2tap_load_snapshot_ex", "h2tap_sync",
+ABI_SYMBOLS = ["h2tap_open", "h2tap_load_snapshot", "h2tap_load_snapshot_ex",
+               "h2tap_load_snapshot_rows", "h2tap_reserve", "h2tap_sync",
                "h2tap_run_query", "h2tap_run_query_ex", "h2tap_run_queries", "h2tap_free", "h2tap_close",
                "h2tap_last_error", "h2tap_nccl_unique_id", "h2tap_compute_stream",
                "h2tap_c_last_name"]
@@ -213,6 +229,43 @@ def h2tap_load_snapshot(engine: Engine, tables: dict, epoch: int, *, flags: int 
     tarr = (h2tap_table * len(tabs))(*tabs)
     _check(_lib.h2tap_load_snapshot_ex(engine.handle, tarr, len(tabs), epoch, flags))
     del keep, colarrs
+
+
+def h2tap_load_snapshot_rows(engine: Engine, tables: dict, epoch: int, *, flags: int = 0,
+                             full_reload=True, first_row: dict | None = None,
+                             columns: dict | None = None) -> None:
+    """Refresh from a host ROW store: ``tables`` = {table_name: numpy structured array of NSM
+    records}. ``columns`` optionally restricts the extracted fields per table (default: every
+    schema field present in the record dtype). Other arguments as h2tap_load_snapshot."""
+    first_row = first_row or {}
+    keep, tabs = [], []
+    for tname, rec in tables.items():
+        tid, schema = SCHEMA[tname]
+        rec = np.ascontiguousarray(rec)
+        want = columns.get(tname) if columns else None
+        fields = []
+        for cid, (cname, ty) in enumerate(schema):
+            if cname not in (rec.dtype.fields or {}) or (want is not None and cname not in want):
+                continue
+            fdt, off = rec.dtype.fields[cname][:2]
+            if fdt != np.dtype(_DT[ty]):
+                raise ValueError(f"{tname}.{cname}: record field {fdt}, schema {np.dtype(_DT[ty])}")
+            fields.append(h2tap_field(cid, ty, off))
+        farr = (h2tap_field * len(fields))(*fields)
+        keep += [rec, farr]
+        full = full_reload if isinstance(full_reload, bool) else tname in full_reload
+        fr = 0 if full else int(first_row.get(tname, 0))
+        tabs.append(h2tap_row_table(tid, len(fields), farr, rec.ctypes.data if len(rec) else None,
+                                    rec.dtype.itemsize, fr + len(rec), fr,
+                                    H2TAP_FULL_RELOAD if full else 0))
+    tarr = (h2tap_row_table * len(tabs))(*tabs)
+    _check(_lib.h2tap_load_snapshot_rows(engine.handle, tarr, len(tabs), epoch, flags))
+    del keep
+
+
+def h2tap_reserve(engine: Engine, table: str, rows: int) -> None:
+    """Pre-size a loaded table's columns for ``rows`` rows (appends then never reallocate)."""
+    _check(_lib.h2tap_reserve(engine.handle, SCHEMA[table][0], rows))
 
 
 def h2tap_sync(engine: Engine) -> int:

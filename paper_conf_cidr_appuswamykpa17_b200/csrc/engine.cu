@@ -21,6 +21,7 @@
 #include <memory>
 #include <mutex>
 #include <string>
+#include <thread>
 #include <vector>
 
 #include <cuda_runtime.h>
@@ -1161,6 +1162,85 @@ h2tap_status h2tap_load_snapshot_ex(h2tap_engine *e, const h2tap_table *tables, 
                                     uint64_t epoch, uint32_t flags) {
     if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
     return guarded([&] { return load_impl(e, tables, ntables, epoch, flags); });
+}
+
+h2tap_status h2tap_reserve(h2tap_engine *e, uint32_t table_id, uint64_t rows) {
+    if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
+    if (table_id < 1 || table_id > 4) return fail(H2TAP_EINVAL, "unknown table id %u", table_id);
+    return guarded([&]() -> h2tap_status {
+        std::lock_guard<std::mutex> g(e->load_mu);
+        CK(cudaSetDevice(e->device));
+        TableState &ts = e->tables[table_id];
+        const uint64_t need = rows + kPadRows;
+        for (int c = 0; c < kNcols[table_id]; ++c) {
+            ColState &cs = ts.col[c];
+            if (!cs.cur || cs.cap_rows >= need) continue;
+            const size_t es = type_size(kTypes[table_id][c]);
+            DevBufP nb = dev_alloc(need * es, e->device);
+            if (ts.loaded)
+                CK(cudaMemcpyAsync(nb->ptr, cs.cur->ptr, ts.loaded * es, cudaMemcpyDeviceToDevice, e->copy));
+            cs.spare.reset();
+            cs.cur = nb;  // published views keep the old buffer alive until they retire
+            cs.cap_rows = need;
+        }
+        CK(cudaStreamSynchronize(e->copy));
+        return H2TAP_OK;
+    });
+}
+
+h2tap_status h2tap_load_snapshot_rows(h2tap_engine *e, const h2tap_row_table *tables,
+                                      uint32_t ntables, uint64_t epoch, uint32_t flags) {
+    if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
+    if (ntables && !tables) return fail(H2TAP_EINVAL, "tables is NULL");
+    return guarded([&]() -> h2tap_status {
+        // column extraction NSM -> DSM into pinned buffers (the library's pinned block pool)
+        std::vector<std::vector<h2tap_column>> cols(ntables);
+        std::vector<h2tap_table> tabs(ntables);
+        std::vector<std::pair<void *, size_t>> blocks;
+        struct Job { const char *src; size_t stride; size_t es; char *dst; uint64_t n; };
+        std::vector<Job> jobs;
+        struct Release {
+            h2tap_engine *e; std::vector<std::pair<void *, size_t>> &b;
+            ~Release() { for (auto &x : b) e->host_pool->put(x.first, x.second); }
+        } release{e, blocks};
+        for (uint32_t t = 0; t < ntables; ++t) {
+            const h2tap_row_table &rt = tables[t];
+            if (rt.row_count < rt.first_row) return fail(H2TAP_EINVAL, "row_count < first_row");
+            const uint64_t n = rt.row_count - rt.first_row;
+            if (n && (!rt.records || !rt.fields)) return fail(H2TAP_EINVAL, "records/fields is NULL");
+            for (uint32_t f = 0; f < rt.nfields; ++f) {
+                const h2tap_field &fd = rt.fields[f];
+                const size_t es = fd.type == H2TAP_I32 ? 4 : 8;
+                if (fd.offset + es > rt.record_size) return fail(H2TAP_EINVAL, "field outside the record");
+                auto b = e->host_pool->get(n * es + 8);
+                blocks.push_back(b);
+                jobs.push_back(Job{static_cast<const char *>(rt.records) + fd.offset, rt.record_size, es,
+                                   static_cast<char *>(b.first), n});
+                cols[t].push_back(h2tap_column{fd.column_id, fd.type, b.first});
+            }
+            tabs[t] = h2tap_table{rt.table_id, rt.nfields, cols[t].data(), rt.row_count, rt.first_row, rt.flags};
+        }
+        // strided gathers, split over host threads by row ranges
+        uint64_t total = 0;
+        for (auto &j : jobs) total += j.n;
+        const unsigned hw = std::max(1u, std::min(16u, std::thread::hardware_concurrency()));
+        const unsigned nthreads = total > (1u << 16) ? hw : 1u;
+        auto work = [&](unsigned tid) {
+            for (auto &j : jobs) {
+                const uint64_t lo = j.n * tid / nthreads, hi = j.n * (tid + 1) / nthreads;
+                if (j.es == 4)
+                    for (uint64_t i = lo; i < hi; ++i) std::memcpy(j.dst + 4 * i, j.src + i * j.stride, 4);
+                else
+                    for (uint64_t i = lo; i < hi; ++i) std::memcpy(j.dst + 8 * i, j.src + i * j.stride, 8);
+            }
+        };
+        std::vector<std::thread> pool;
+        for (unsigned t = 1; t < nthreads; ++t) pool.emplace_back(work, t);
+        work(0);
+        for (auto &th : pool) th.join();
+        // pinned sources: load_impl DMAs them directly and waits before returning
+        return load_impl(e, tabs.data(), ntables, epoch, flags);
+    });
 }
 
 h2tap_status h2tap_load_snapshot(h2tap_engine *e, const h2tap_table *tables, uint32_t ntables,

@@ -358,6 +358,32 @@ def test_snapshot_epochs_append_and_errors(h):
         h.h2tap_close(e)
 
 
+def test_row_store_refresh(h):
+    """h2tap_load_snapshot_rows: NSM records -> DSM snapshot (full load, then an append)."""
+    e = h.h2tap_open(0)
+    try:
+        base = chgen.generate(1, 3, seed=33)
+        cols = {tb: list(c) for tb, c in h.hot_path_tables(base).items()}
+        recs = {tb: chgen.to_records(tb, base[tb]) for tb in ("order_line", "orders", "customer")}
+        h.h2tap_load_snapshot_rows(e, recs, 1, columns=cols)
+        r = h.h2tap_run_query(e, h.H2TAP_Q18, [-1]); got = r.to_numpy(); r.free()
+        assert_q18(got, oracle.q18(base, -1))
+        st = chgen.NewOrderState(1, 3)
+        d = chgen.neworder_batch(st, 500, seed=33, batch=0, item=base["item"])
+        drec = {tb: chgen.to_records(tb, d[tb]) for tb in ("order_line", "orders")}
+        h.h2tap_load_snapshot_rows(e, drec, 2, full_reload=False, columns=cols,
+                                   first_row={tb: len(recs[tb]) for tb in drec})
+        merged = {tb: {c: np.concatenate([base[tb][c], d[tb][c]]) for c in base[tb]}
+                  for tb in ("order_line", "orders")}
+        merged["customer"] = base["customer"]
+        r = h.h2tap_run_query(e, h.H2TAP_Q18, [-1]); got = r.to_numpy(); r.free()
+        assert_q18(got, oracle.q18(merged, -1))
+        r = h.h2tap_run_query(e, h.H2TAP_Q1); got = r.to_numpy(); r.free()
+        assert_q1(got, oracle.q1(merged, Q1_CUTOFF))
+    finally:
+        h.h2tap_close(e)
+
+
 def test_concurrent_refresh_and_queries(h):
     """Queries running while another thread appends see a consistent published epoch."""
     import threading
