@@ -785,10 +785,26 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     e->prof.run("q18_sort_keys", [&] {
         launch_q18_sort_keys(q.rows, q.amt, q.plan_dev, n_max, q.sp, e->num_sms, e->compute);
     });
-    e->prof.run("q18_bucket_sort", [&] {
-        bucket_sort_pairs(n_max, &q.plan_dev->n, &q.plan_dev->shift, bb, bs, q.tie_dev, e->num_sms,
-                          e->compute);
-    });
+    struct Marks : PhaseMarks {  // one profile mark per bucket-sort kernel
+        Prof &p;
+        cudaEvent_t a = nullptr;
+        std::string name;
+        explicit Marks(Prof &pr) : p(pr) {}
+        void begin(const char *nm) override {
+            if (!p.on) return;
+            name = nm;
+            a = p.ev();
+            CK(cudaEventRecord(a, p.st));
+        }
+        void end() override {
+            if (!p.on) return;
+            cudaEvent_t b = p.ev();
+            CK(cudaEventRecord(b, p.st));
+            p.marks.push_back({name, {a, b}});
+        }
+    } marks(e->prof);
+    bucket_sort_pairs(n_max, &q.plan_dev->n, &q.plan_dev->shift, bb, bs, q.tie_dev, e->num_sms,
+                      e->compute, &marks);
     e->prof.run("q18_tiefix", [&] {
         launch_q18_tiefix(q.rows, q.amt, q.sp.k[1], q.sp.v[1], q.plan_dev, n_max, q.tie_dev,
                           e->num_sms, e->compute);

@@ -138,9 +138,15 @@ struct BucketSort {
 // Sorted pairs end in k[1]/v[1] (input in k[0]/v[0]). The row count and the bucket shift are
 // read on the device (*dn, *dshift), so the whole ORDER BY runs without a host round trip;
 // `n_max` (an upper bound of *dn) only sizes the grids.
+// Optional per-kernel profiling marks (the engine records CUDA events around each phase).
+struct PhaseMarks {
+    virtual void begin(const char *name) = 0;
+    virtual void end() = 0;
+    virtual ~PhaseMarks() = default;
+};
 void bucket_sort_pairs(uint64_t n_max, const unsigned long long *dn, const int *dshift,
                        int bucket_bits, const BucketSort &s, unsigned int *flag, int num_sms,
-                       cudaStream_t st);
+                       cudaStream_t st, PhaseMarks *marks = nullptr);
 
 // Q18 ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id (R11).
 struct Q18SortSpec {         // host-computed from Q18Stats

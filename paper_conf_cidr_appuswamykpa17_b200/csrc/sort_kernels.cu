@@ -621,7 +621,9 @@ bucket_local_sort_kernel(unsigned long long *__restrict__ k, unsigned int *__res
 
 void bucket_sort_pairs(uint64_t n_max, const unsigned long long *dn, const int *dshift,
                        int bucket_bits, const BucketSort &s, unsigned int *flag, int num_sms,
-                       cudaStream_t st) {
+                       cudaStream_t st, PhaseMarks *marks) {
+    auto begin = [&](const char *nm) { if (marks) marks->begin(nm); };
+    auto end = [&] { if (marks) marks->end(); };
     if (bucket_bits > kBucketMaxBits) bucket_bits = kBucketMaxBits;
     const int nb = 1 << bucket_bits;
     static bool init = false;
@@ -642,23 +644,33 @@ void bucket_sort_pairs(uint64_t n_max, const unsigned long long *dn, const int *
     uint64_t hb = (n_max + per - 1) / per;
     if (hb > (uint64_t)num_sms * 2) hb = (uint64_t)num_sms * 2;
     if (!hb) hb = 1;
+    begin("q18_bucket_hist");
     bucket_hist_kernel<<<(unsigned)hb, kBkThreads, nb * 4, st>>>(s.k[0], dn, dshift, nb, s.count);
     count_launches(1);
+    end();
+    begin("q18_bucket_scan");
     bucket_scan_kernel<<<1, 1024, 0, st>>>(s.count, nb, s.offset, s.cursor);
     count_launches(1);
+    end();
+    begin("q18_bucket_scatter");
     const uint64_t sb = (n_max + per - 1) / per;
     bucket_scatter_kernel<<<(unsigned)(sb ? sb : 1), kBkThreads, nb * 4, st>>>(
         s.k[0], s.v[0], s.k[1], s.v[1], dn, dshift, nb, s.cursor);
     count_launches(1);
+    end();
+    begin("q18_bucket_local");
     unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
     bucket_local_sort_kernel<kLsCapSmall, 0><<<lb, kBkThreads, sizeof(LsSmem<kLsCapSmall>), st>>>(
         s.k[1], s.v[1], s.offset, nb, dshift, flag, s.big);
     count_launches(1);
+    end();
     // buckets above the small capacity (skewed keys): one block per SM, ~200 KB shared memory
+    begin("q18_bucket_local_large");
     bucket_local_sort_kernel<kLsCapLarge, kLsCapSmall><<<(unsigned)num_sms, kBkThreads,
                                                           sizeof(LsSmem<kLsCapLarge>), st>>>(
         s.k[1], s.v[1], s.offset, nb, dshift, flag, s.big);
     count_launches(1);
+    end();
 }
 
 }  // namespace h2tap

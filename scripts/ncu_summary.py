@@ -60,10 +60,15 @@ if traffic:
              "q18_init_kernel": "q18_init", "q18_build_kernel": "q18_build",
              "q18_probe_kernel": "q18_probe_groupjoin", "q18_having_kernel": "q18_having_compact",
              "sort_keys_kernel": "q18_sort_keys", "tiefix_kernel": "q18_tiefix",
-             "permute_kernel": "q18_permute"}
+             "permute_kernel": "q18_permute", "bucket_hist_kernel": "q18_bucket_hist",
+             "bucket_scan_kernel": "q18_bucket_scan", "bucket_scatter_kernel": "q18_bucket_scatter",
+             "bucket_local_sort_kernel<2048, 0>": "q18_bucket_local",
+             "bucket_local_sort_kernel<8192, 2048>": "q18_bucket_local_large",
+             "q18_plan_kernel": "q18_plan", "q1_compact_kernel": "q1_compact",
+             "q1_emit_kernel": "q1_emit"}
     bymark = {}
     for k, v in per.items():
-        m = marks.get(k, "q18_bucket_sort" if k.startswith("bucket_") else None)
+        m = marks.get(k)
         if m:
             bymark[m] = bymark.get(m, 0.0) + v
     if len(sys.argv) > 2 and sys.argv[2] == "--bench":

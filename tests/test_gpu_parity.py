@@ -273,7 +273,7 @@ def test_profile_reports_kernels(h, eng, L):
     L.load(t)
     r = h.h2tap_run_query(eng, h.H2TAP_Q18, flags=h.H2TAP_QUERY_PROFILE)
     names = [k for k, _ in r.kernels]
-    assert {"q18_build", "q18_probe_groupjoin", "q18_having_compact", "q18_bucket_sort"} <= set(names)
+    assert {"q18_build", "q18_probe_groupjoin", "q18_having_compact", "q18_bucket_scatter", "q18_bucket_local"} <= set(names)
     assert all(ms >= 0 for _, ms in r.kernels) and r.device_ms > 0
     r.free()
 
@@ -368,6 +368,8 @@ def test_row_store_refresh(h):
         h.h2tap_load_snapshot_rows(e, recs, 1, columns=cols)
         r = h.h2tap_run_query(e, h.H2TAP_Q18, [-1]); got = r.to_numpy(); r.free()
         assert_q18(got, oracle.q18(base, -1))
+        h.h2tap_reserve(e, "order_line", len(recs["order_line"]) + 100_000)  # pre-size, then append
+        h.h2tap_reserve(e, "orders", len(recs["orders"]) + 10_000)
         st = chgen.NewOrderState(1, 3)
         d = chgen.neworder_batch(st, 500, seed=33, batch=0, item=base["item"])
         drec = {tb: chgen.to_records(tb, d[tb]) for tb in ("order_line", "orders")}
@@ -480,5 +482,19 @@ def test_full_size_w100_bench_config(h, w100):
         want = oracle.q18(w100, Q18_HAVING)
         assert_q18(L.q(18, flags=h.H2TAP_QUERY_PROFILE), want)
         assert_q18(L.q(18, flags=HASH), want)
+    finally:
+        h.h2tap_close(e)
+
+
+def test_full_size_w100_strict(h):
+    """W=100 with the strict TPC-C population: 64-bit exact composite ORDER BY path."""
+    t = chgen.generate(1, 101, seed=2, mode="strict")
+    e = h.h2tap_open(0)
+    try:
+        h.h2tap_load_snapshot(e, h.hot_path_tables(t), 1)
+        L = Loader(h, e)
+        assert_q6(L.q(6), oracle.q6(t, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))
+        assert_q1(L.q(1), oracle.q1(t, Q1_CUTOFF))
+        assert_q18(L.q(18), oracle.q18(t, Q18_HAVING))
     finally:
         h.h2tap_close(e)
