@@ -134,12 +134,9 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes):
         "q18_build": 12 * n_o + 12 * n_c + 16 * (n_o + n_c),
         "q18_probe_groupjoin": 20 * n_ol + 16 * n_o + 16 * n_o,
         "q18_having_compact": 16 * n_o + 28 * n_o + 16 * n_pass + 4 * n_pass + 40 * n_pass,
-        "q18_sort_keys": 40 * n_pass + 24 * n_pass,
-        "q18_bucket_hist": 8 * n_pass,                 # read keys
-        "q18_bucket_scatter": (12 + 12) * n_pass,      # read + write (key, row id)
-        "q18_bucket_local": (12 + 12) * n_pass,        # read + write (key, row id) per bucket
-        "q18_tiefix": 8 * n_pass,
-        "q18_permute": (4 + 40 + 40) * n_pass,
+        "q18_sort_keys_hist": (32 + 8 + 8 + 4) * n_pass,   # rows + amounts -> keys + row ids
+        "q18_bucket_scatter": (12 + 12) * n_pass,          # read + write (key, row id)
+        "q18_bucket_sort_emit": (12 + 32 + 40) * n_pass,   # (key, id), row gather, 8 result columns
     }.get(kernel)
 
 

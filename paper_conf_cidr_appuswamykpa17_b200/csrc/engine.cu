@@ -761,8 +761,9 @@ struct Q18Small { unsigned long long nout; unsigned int err, tie; Q18Stats st; }
 
 void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     // a8: ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id, entirely on the device:
-    // plan (field widths from the stats) -> 64-bit prefix keys -> bucket sort -> tie-fix ->
-    // gather into the output columns. Grids are sized for n_max (the orders rows).
+    // plan (field widths from the stats) -> 64-bit prefix keys + bucket histogram -> bucket
+    // scatter -> per-bucket sort + tie-fix + emit into the output columns. Grids are sized for
+    // n_max (the orders rows); the actual row count is read on the device.
     const uint64_t n_max = std::max<uint64_t>(q.n_max, 1);
     int bb = 1;
     while (bb < kBucketMaxBits && (n_max >> (bb + 9)) > 0) ++bb;   // ~256-512 rows per bucket
@@ -780,12 +781,19 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     bs.cursor = static_cast<unsigned int *>(e->arena.get("q18.bcursor", 4 * (1 << kBucketMaxBits)));
     bs.offset = static_cast<unsigned int *>(e->arena.get("q18.boffset", 4 * ((1 << kBucketMaxBits) + 1)));
     bs.big = static_cast<unsigned int *>(e->arena.get("q18.bbig", 4 * ((1 << kBucketMaxBits) + 1)));
+    bs.ticket = static_cast<unsigned int *>(e->arena.get("q18.bticket", 64, true, e->compute));
     q.tie_dev = static_cast<unsigned int *>(e->arena.get("q18.tie", 64));
     CK(cudaMemsetAsync(q.tie_dev, 0, 4, e->compute));
-    e->prof.run("q18_sort_keys", [&] {
-        launch_q18_sort_keys(q.rows, q.amt, q.plan_dev, n_max, q.sp, e->num_sms, e->compute);
-    });
-    struct Marks : PhaseMarks {  // one profile mark per bucket-sort kernel
+    Q18Cols &d = q.out;
+    d.c_last = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    d.c_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    d.o_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    d.o_entry_d = static_cast<int64_t *>(dev_block(e, q, 8 * n_max));
+    d.o_ol_cnt = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    d.amount_sum = static_cast<int64_t *>(dev_block(e, q, 8 * n_max));
+    d.o_w_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    d.o_d_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
+    struct Marks : PhaseMarks {  // one profile mark per ORDER BY kernel
         Prof &p;
         cudaEvent_t a = nullptr;
         std::string name;
@@ -803,26 +811,8 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
             p.marks.push_back({name, {a, b}});
         }
     } marks(e->prof);
-    bucket_sort_pairs(n_max, &q.plan_dev->n, &q.plan_dev->shift, bb, bs, q.tie_dev, e->num_sms,
-                      e->compute, &marks);
-    e->prof.run("q18_tiefix", [&] {
-        launch_q18_tiefix(q.rows, q.amt, q.sp.k[1], q.sp.v[1], q.plan_dev, n_max, q.tie_dev,
-                          e->num_sms, e->compute);
-    });
-    q.perm = q.sp.v[1];
-    q.perm_keys = q.sp.k[1];
-    Q18Cols &d = q.out;
-    d.c_last = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    d.c_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    d.o_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    d.o_entry_d = static_cast<int64_t *>(dev_block(e, q, 8 * n_max));
-    d.o_ol_cnt = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    d.amount_sum = static_cast<int64_t *>(dev_block(e, q, 8 * n_max));
-    d.o_w_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    d.o_d_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    e->prof.run("q18_permute", [&] {
-        launch_q18_permute(q.rows, q.amt, q.perm, q.perm_keys, q.plan_dev, n_max, d, e->num_sms, e->compute);
-    });
+    q18_bucket_order(q.rows, q.amt, q.plan_dev, n_max, bb, bs, d, q.tie_dev, e->num_sms, e->compute,
+                     &marks);
 }
 
 void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
@@ -1155,6 +1145,7 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
             return fail(H2TAP_ECUDA, "built for sm_100a (B200); device %d is sm_%d%d", e->device,
                         prop.major, prop.minor);
         e->num_sms = prop.multiProcessorCount;
+
         CK(cudaStreamCreateWithFlags(&e->compute, cudaStreamNonBlocking));
         CK(cudaStreamCreateWithFlags(&e->copy, cudaStreamNonBlocking));
         CK(cudaEventCreate(&e->q_begin));

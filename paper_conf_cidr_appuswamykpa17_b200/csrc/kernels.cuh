@@ -122,10 +122,9 @@ struct SortPairs {
 // Returns which buffer (0/1) holds the sorted pairs (input is in k[0]/v[0]).
 int radix_sort_pairs(uint64_t n, int bits, const SortPairs &s, int num_sms, cudaStream_t st);
 
-// Bucket sort of (u64 key, u32 value) pairs whose keys use the low `bits` bits: partition by the
-// top `bucket_bits` key bits (histogram -> scan -> scatter), then sort every bucket in shared
-// memory (two-level: sub-buckets + rank). A bucket larger than 4096 rows raises *flag (the caller
-// falls back to the exact LSD sort).
+// Scratch of the ORDER BY bucket sort: keys + row ids ping-pong, bucket counts,
+// offsets/cursors, a work list of buckets above the small in-shared-memory capacity, and the
+// last-block ticket of the keys+histogram kernel.
 constexpr int kBucketMaxBits = 15;
 struct BucketSort {
     unsigned long long *k[2];
@@ -134,19 +133,14 @@ struct BucketSort {
     unsigned int *cursor;  // [2^kBucketMaxBits]
     unsigned int *offset;  // [2^kBucketMaxBits + 1]
     unsigned int *big;     // [1 + 2^kBucketMaxBits]: count, then ids of buckets > small capacity
+    unsigned int *ticket;  // [1], zero-initialised once, self-resetting
 };
-// Sorted pairs end in k[1]/v[1] (input in k[0]/v[0]). The row count and the bucket shift are
-// read on the device (*dn, *dshift), so the whole ORDER BY runs without a host round trip;
-// `n_max` (an upper bound of *dn) only sizes the grids.
 // Optional per-kernel profiling marks (the engine records CUDA events around each phase).
 struct PhaseMarks {
     virtual void begin(const char *name) = 0;
     virtual void end() = 0;
     virtual ~PhaseMarks() = default;
 };
-void bucket_sort_pairs(uint64_t n_max, const unsigned long long *dn, const int *dshift,
-                       int bucket_bits, const BucketSort &s, unsigned int *flag, int num_sms,
-                       cudaStream_t st, PhaseMarks *marks = nullptr);
 
 // Q18 ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id (R11).
 struct Q18SortSpec {         // host-computed from Q18Stats
@@ -167,12 +161,13 @@ struct Q18Plan {
 };
 void launch_q18_plan(const Q18Stats *stats, const unsigned long long *nout, int bucket_bits,
                      Q18Plan *plan, cudaStream_t st);
-void launch_q18_sort_keys(const Q18Row *rows, const long long *amt, const Q18Plan *plan,
-                          uint64_t n_max, const SortPairs &s, int num_sms, cudaStream_t st);
+// The whole ORDER BY: keys + histogram -> bucket scatter -> per-bucket sort, tie-fix and emit
+// into `dst` (final positions). Everything reads the row count and widths from *plan.
+// *flag: bit0 a tie run > 32 rows, bit1 a bucket > 8192 rows (caller redoes it exactly).
+void q18_bucket_order(const Q18Row *rows, const long long *amt, const Q18Plan *plan, uint64_t n_max,
+                      int bucket_bits, const BucketSort &s, const Q18Cols &dst, unsigned int *flag,
+                      int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr);
 // Within runs of equal prefix, order by the full tuple; runs longer than 32 raise *flag.
-void launch_q18_tiefix(const Q18Row *rows, const long long *amt, const unsigned long long *keys,
-                       unsigned int *vals, const Q18Plan *plan, uint64_t n_max, unsigned int *flag,
-                       int num_sms, cudaStream_t st);
 // Exact fallback: three stable passes over the full fields (row rank, entry, amount).
 void launch_q18_field_keys(const Q18Row *rows, const long long *amt, const unsigned int *vals,
                            uint64_t n, int field, const Q18Plan *plan, unsigned long long *keys,

@@ -186,18 +186,6 @@ __device__ __forceinline__ unsigned long long prefix_key(const Q18Row &r, long l
     return p;
 }
 
-__global__ void sort_keys_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
-                                 const Q18Plan *__restrict__ plan, unsigned long long *__restrict__ k,
-                                 unsigned int *__restrict__ v) {
-    const uint64_t n = plan->n;
-    const Q18SortSpec sp = plan->spec;
-    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
-        k[i] = prefix_key(rows[i], amt[i], sp);
-        v[i] = (unsigned int)i;
-    }
-}
-
 // full ORDER BY comparison: amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id
 __device__ __forceinline__ bool row_less(const Q18Row &x, long long ax, const Q18Row &y, long long ay) {
     if (ax != ay) return ax > ay;
@@ -208,34 +196,6 @@ __device__ __forceinline__ bool row_less(const Q18Row &x, long long ax, const Q1
 }
 
 constexpr int kMaxRun = 32;
-
-__global__ void tiefix_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
-                              const unsigned long long *__restrict__ k, unsigned int *__restrict__ v,
-                              const Q18Plan *__restrict__ plan, unsigned int *flag) {
-    if (!plan->tiefix) return;  // composite key fits 64 bits: keys are distinct
-    const uint64_t n = plan->n;
-    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
-        const unsigned long long ki = k[i];
-        if (i > 0 && k[i - 1] == ki) continue;         // not the head of a run
-        if (i + 1 >= n || k[i + 1] != ki) continue;    // run of one
-        uint64_t j = i + 1;
-        while (j < n && k[j] == ki && j - i <= kMaxRun) ++j;
-        if (j - i > kMaxRun) { atomicOr(flag, 1u); continue; }
-        unsigned int idx[kMaxRun];
-        const int len = (int)(j - i);
-        for (int t = 0; t < len; ++t) idx[t] = v[i + t];
-        for (int t = 1; t < len; ++t) {  // insertion sort by the full tuple
-            const unsigned int x = idx[t];
-            const Q18Row rx = rows[x];
-            const long long ax = amt[x];
-            int u = t - 1;
-            while (u >= 0 && row_less(rx, ax, rows[idx[u]], amt[idx[u]])) { idx[u + 1] = idx[u]; --u; }
-            idx[u + 1] = x;
-        }
-        for (int t = 0; t < len; ++t) v[i + t] = idx[t];
-    }
-}
 
 __global__ void field_keys_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
                                   const unsigned int *__restrict__ vals, uint64_t n, int field,
@@ -352,19 +312,6 @@ int radix_sort_pairs(uint64_t n, int bits, const SortPairs &s, int num_sms, cuda
     return cur;
 }
 
-void launch_q18_sort_keys(const Q18Row *rows, const long long *amt, const Q18Plan *plan,
-                          uint64_t n_max, const SortPairs &s, int num_sms, cudaStream_t st) {
-    sort_keys_kernel<<<grid_cap(n_max, 256, num_sms, 8), 256, 0, st>>>(rows, amt, plan, s.k[0], s.v[0]);
-    count_launches(1);
-}
-
-void launch_q18_tiefix(const Q18Row *rows, const long long *amt, const unsigned long long *keys,
-                       unsigned int *vals, const Q18Plan *plan, uint64_t n_max, unsigned int *flag,
-                       int num_sms, cudaStream_t st) {
-    tiefix_kernel<<<grid_cap(n_max, 256, num_sms, 8), 256, 0, st>>>(rows, amt, keys, vals, plan, flag);
-    count_launches(1);
-}
-
 void launch_q18_field_keys(const Q18Row *rows, const long long *amt, const unsigned int *vals,
                            uint64_t n, int field, const Q18Plan *plan, unsigned long long *keys,
                            int num_sms, cudaStream_t st) {
@@ -387,113 +334,114 @@ void launch_q18_permute(const Q18Row *rows, const long long *amt, const unsigned
 }  // namespace h2tap
 
 // ============================================================ bucket sort ===
-// Main ORDER BY path: the result (a few million 12-byte pairs) fits in L2, so
-// one partition pass by the top key bits plus a shared-memory sort per bucket replaces LSD
-// passes. Inside a bucket: a second partition by the next bits into sub-buckets of ~8 rows, then
-// every row's final position is its rank inside its sub-bucket (count of smaller keys, ties by
-// position) — no barriers inside the ranking. Equal 64-bit prefixes are ordered afterwards by
-// the tie-fix kernel (full tuple), so the result is the same total order as the LSD path.
+// Main ORDER BY path, three kernels:
+//  1. keys+hist: the 64-bit prefix key of every result row, the row id, a shared-memory
+//     histogram of the top key bits; the last block to finish scans the bucket counts;
+//  2. scatter: rows into buckets (per-block range reservation, shared cursors);
+//  3. local sort + emit: each bucket in shared memory — second partition into ~8-row sub-buckets
+//     and rank counting, then runs of equal prefixes ordered by the full tuple (tie-fix), then
+//     the rows are gathered and written straight into the result columns at their final
+//     positions (amount_sum decoded from the key).
+// A bucket > 8192 rows or a tie run > 32 rows sets *flag; the engine then redoes the ORDER BY
+// exactly with the LSD fallback above.
 namespace h2tap {
 namespace {
 
 constexpr int kBkThreads = 256;
-constexpr int kBkItems = 16;                       // rows per thread in hist/scatter
+constexpr int kBkItems = 16;                       // rows per thread in the scatter
 constexpr int kLsCapSmall = 2048;                  // rows per bucket: fast kernel (3 blocks/SM)
 constexpr int kLsCapLarge = 8192;                  // rows per bucket: large-bucket kernel
 constexpr int kLsSubMax = 1024;                    // max sub-buckets per bucket
 
+// 1. keys + histogram (+ bucket scan by the last block)
 __global__ void __launch_bounds__(kBkThreads)
-bucket_hist_kernel(const unsigned long long *__restrict__ key, const unsigned long long *dn,
-                   const int *dshift, int nb, unsigned int *__restrict__ count) {
-    const uint64_t n = *dn;
-    const int shift = *dshift;
+q18_keys_hist_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
+                     const Q18Plan *__restrict__ plan, unsigned long long *__restrict__ k,
+                     unsigned int *__restrict__ v, int nb, unsigned int *__restrict__ count,
+                     unsigned int *__restrict__ offset, unsigned int *__restrict__ cursor,
+                     unsigned int *ticket) {
     extern __shared__ unsigned int h[];
+    __shared__ bool last;
+    __shared__ unsigned int wsum[kBkThreads / 32];
+    const uint64_t n = plan->n;
+    const Q18SortSpec sp = plan->spec;
+    const int shift = plan->shift;
     for (int i = threadIdx.x; i < nb; i += kBkThreads) h[i] = 0;
     __syncthreads();
-    for (uint64_t base = (uint64_t)blockIdx.x * kBkThreads * kBkItems; base < n;
-         base += (uint64_t)gridDim.x * kBkThreads * kBkItems) {
-        unsigned int b[kBkItems];
+    const uint64_t stride = (uint64_t)gridDim.x * kBkThreads;
+    constexpr int U = 4;  // independent row loads in flight per thread
+    for (uint64_t i0 = (uint64_t)blockIdx.x * kBkThreads + threadIdx.x; i0 < n; i0 += U * stride) {
+        Q18Row r[U];
+        long long a[U];
 #pragma unroll
-        for (int i = 0; i < kBkItems; ++i) {
-            const uint64_t j = base + (uint64_t)i * kBkThreads + threadIdx.x;
-            b[i] = j < n ? (unsigned int)(__ldcg(key + j) >> shift) : 0xffffffffu;
+        for (int u = 0; u < U; ++u) {
+            const uint64_t i = i0 + u * stride;
+            if (i < n) { r[u] = rows[i]; a[u] = amt[i]; }
         }
 #pragma unroll
-        for (int i = 0; i < kBkItems; ++i)
-            if (b[i] != 0xffffffffu) atomicAdd(&h[b[i]], 1u);
+        for (int u = 0; u < U; ++u) {
+            const uint64_t i = i0 + u * stride;
+            if (i >= n) break;
+            const unsigned long long kk = prefix_key(r[u], a[u], sp);
+            k[i] = kk;
+            v[i] = (unsigned int)i;
+            atomicAdd(&h[(unsigned int)(kk >> shift)], 1u);
+        }
     }
     __syncthreads();
     for (int i = threadIdx.x; i < nb; i += kBkThreads)
         if (h[i]) atomicAdd(count + i, h[i]);
-}
-
-// exclusive scan of nb (<= 32768) bucket counts -> offset[] and cursor[]; one pass: each of
-// 1024 threads owns nb/1024 contiguous counts (all loads issued first); max size -> count[nb]
-__global__ void __launch_bounds__(1024) bucket_scan_kernel(unsigned int *__restrict__ count, int nb,
-                                                           unsigned int *__restrict__ offset,
-                                                           unsigned int *__restrict__ cursor) {
-    __shared__ unsigned int wsum[32], wmax[32];
+    __threadfence();
+    __syncthreads();
+    if (threadIdx.x == 0) last = atomicAdd(ticket, 1u) == gridDim.x - 1;
+    __syncthreads();
+    if (!last) return;
+    __threadfence();
+    // exclusive scan of the nb bucket counts: each thread owns nb/256 contiguous counts
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    const int per = (nb + 1023) / 1024;  // <= 32
+    const int per = (nb + kBkThreads - 1) / kBkThreads;
     const int b0 = threadIdx.x * per;
-    unsigned int t = 0, mx = 0;
-#pragma unroll 8
-    for (int q = 0; q < per; ++q) {  // pass 1: chunk total (re-read in pass 2 from L2)
-        const unsigned int c = b0 + q < nb ? count[b0 + q] : 0u;
-        t += c;
-        mx = max(mx, c);
-    }
+    unsigned int t = 0;
+    for (int q = 0; q < per && b0 + q < nb; ++q) t += __ldcg(count + b0 + q);
     unsigned int x = t;
 #pragma unroll
     for (int o = 1; o < 32; o <<= 1) {
         const unsigned int y = __shfl_up_sync(kFull, x, o);
         if (lane >= o) x += y;
     }
-    mx = __reduce_max_sync(kFull, mx);
     if (lane == 31) wsum[warp] = x;
-    if (lane == 0) wmax[warp] = mx;
     __syncthreads();
-    unsigned int before = 0, total = 0, m = 0;
-    for (int w = 0; w < 32; ++w) {
-        before += w < warp ? wsum[w] : 0u;
-        total += wsum[w];
-        m = max(m, wmax[w]);
-    }
-    unsigned int run = before + x - t;
-#pragma unroll 8
-    for (int q = 0; q < per; ++q) {
-        if (b0 + q >= nb) break;
-        const unsigned int c = count[b0 + q];
+    unsigned int run = x - t;
+    for (int w = 0; w < warp; ++w) run += wsum[w];
+    for (int q = 0; q < per && b0 + q < nb; ++q) {
+        const unsigned int c = __ldcg(count + b0 + q);
         offset[b0 + q] = run;
         cursor[b0 + q] = run;
         run += c;
     }
-    if (threadIdx.x == 0) {
-        offset[nb] = total;
-        count[nb] = m;
-    }
+    if (threadIdx.x == kBkThreads - 1) offset[nb] = run;
+    if (threadIdx.x == 0) *ticket = 0;  // self-reset for the next launch
 }
 
-// scatter into buckets: a block's shared histogram reserves one global range per bucket
+// 2. scatter into buckets: a block's shared histogram reserves one global range per bucket
 __global__ void __launch_bounds__(kBkThreads)
 bucket_scatter_kernel(const unsigned long long *__restrict__ kin, const unsigned int *__restrict__ vin,
                       unsigned long long *__restrict__ kout, unsigned int *__restrict__ vout,
-                      const unsigned long long *dn, const int *dshift, int nb,
-                      unsigned int *__restrict__ cursor) {
-    const uint64_t n = *dn;
-    const int shift = *dshift;
+                      const Q18Plan *__restrict__ plan, int nb, unsigned int *__restrict__ cursor) {
+    const uint64_t n = plan->n;
+    const int shift = plan->shift;
     if ((uint64_t)blockIdx.x * kBkThreads * kBkItems >= n) return;  // grid sized for an upper bound
     extern __shared__ unsigned int h[];  // [nb] local counts -> local cursors
     for (int i = threadIdx.x; i < nb; i += kBkThreads) h[i] = 0;
     const uint64_t base = (uint64_t)blockIdx.x * kBkThreads * kBkItems;
-    unsigned long long k[kBkItems];
+    unsigned long long kv[kBkItems];
     unsigned int b[kBkItems], val[kBkItems];
 #pragma unroll
     for (int i = 0; i < kBkItems; ++i) {
         const uint64_t j = base + (uint64_t)i * kBkThreads + threadIdx.x;
-        k[i] = j < n ? __ldcs(kin + j) : 0ull;
+        kv[i] = j < n ? __ldcs(kin + j) : 0ull;
         val[i] = j < n ? __ldcs(vin + j) : 0u;
-        b[i] = j < n ? (unsigned int)(k[i] >> shift) : 0xffffffffu;
+        b[i] = j < n ? (unsigned int)(kv[i] >> shift) : 0xffffffffu;
     }
     __syncthreads();
 #pragma unroll
@@ -511,7 +459,7 @@ bucket_scatter_kernel(const unsigned long long *__restrict__ kin, const unsigned
 #pragma unroll
     for (int i = 0; i < kBkItems; ++i) {
         if (b[i] == 0xffffffffu) continue;
-        kout[pos[i]] = k[i];
+        kout[pos[i]] = kv[i];
         vout[pos[i]] = val[i];
     }
 }
@@ -524,25 +472,30 @@ template <int kLsCap> struct LsSmem {
     unsigned int wsum[kBkThreads / 32];
 };
 
-// One block per bucket: load it into shared memory, partition by the next `sb` key bits into
-// sub-buckets, write every row at offset + its rank within its sub-bucket. The kernel handles
-// buckets of (kMin, kLsCap] rows; the large instance flags buckets above its capacity.
+// 3. One block per bucket: partition by the next `sb` key bits into sub-buckets, rank every row
+// inside its sub-bucket, order equal-prefix runs by the full tuple, and write the result columns
+// at their final positions. The small instance walks every bucket and queues buckets above its
+// capacity in big[1..]; the large instance walks only that queue.
 template <int kLsCap, int kMin>
 __global__ void __launch_bounds__(kBkThreads)
-bucket_local_sort_kernel(unsigned long long *__restrict__ k, unsigned int *__restrict__ v,
-                         const unsigned int *__restrict__ offset, int nb, const int *dshift,
-                         unsigned int *flag, unsigned int *big) {
-    const int shift = *dshift;
+bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigned int *__restrict__ v,
+                         const unsigned int *__restrict__ offset, int nb,
+                         const Q18Plan *__restrict__ plan, const Q18Row *__restrict__ rows,
+                         const long long *__restrict__ amt, Q18Cols dst, unsigned int *flag,
+                         unsigned int *big) {
     extern __shared__ __align__(16) unsigned char smem_raw[];
     LsSmem<kLsCap> &S = *reinterpret_cast<LsSmem<kLsCap> *>(smem_raw);
+    const int shift = plan->shift;
+    const Q18SortSpec sp = plan->spec;
+    const bool tiefix = plan->tiefix != 0;
+    const int ashift = sp.prefix_bits - sp.bits_a;
+    const uint64_t drop = l2_policy_evict_first();  // last read of the result rows
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    // the small instance walks every bucket and queues the big ones in big[1..]; the large
-    // instance walks only that queue
     const int nwork = kMin > 0 ? (int)*(volatile unsigned int *)big : nb;
     for (int wi = blockIdx.x; wi < nwork; wi += gridDim.x) {
         const int b = kMin > 0 ? (int)big[1 + wi] : wi;
         const unsigned int lo = offset[b], m = offset[b + 1] - lo;
-        if (m <= 1) continue;
+        if (m == 0) continue;
         if (m > (unsigned)kLsCap) {
             if (threadIdx.x == 0) {
                 if (kMin > 0) atomicOr(flag, 2u);                 // too big even for shared memory
@@ -550,68 +503,115 @@ bucket_local_sort_kernel(unsigned long long *__restrict__ k, unsigned int *__res
             }
             continue;
         }
-        // sub-bucket bits: ~8 rows per sub-bucket, at most kLsSubMax sub-buckets
-        int sb = 0;
-        while (sb < 10 && (m >> (sb + 3)) > 0) ++sb;
-        if (sb > shift) sb = shift;
-        const int ssh = shift - sb;
-        const unsigned int ns = 1u << sb, smask = ns - 1u;
-        for (unsigned int i = threadIdx.x; i < ns; i += kBkThreads) S.sub[i] = 0;
-        __syncthreads();
-        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
-            const unsigned long long kk = k[lo + i];
-            S.k1[i] = kk;
-            S.v1[i] = v[lo + i];
-            atomicAdd(&S.sub[(unsigned int)(kk >> ssh) & smask], 1u);
-        }
-        __syncthreads();
-        // exclusive scan of ns (<= 1024) sub-bucket counts: 4 per thread
-        {
-            unsigned int c[4], t = 0;
-#pragma unroll
-            for (int q = 0; q < 4; ++q) {
-                const unsigned int i = threadIdx.x * 4 + q;
-                c[q] = i < ns ? S.sub[i] : 0u;
-                t += c[q];
-            }
-            unsigned int x = t;
-#pragma unroll
-            for (int o = 1; o < 32; o <<= 1) {
-                const unsigned int y = __shfl_up_sync(kFull, x, o);
-                if (lane >= o) x += y;
-            }
-            if (lane == 31) S.wsum[warp] = x;
+        if (m == 1) {
+            if (threadIdx.x == 0) { S.k1[0] = k[lo]; S.v1[0] = v[lo]; }
+        } else {
+            // sub-bucket bits: ~8 rows per sub-bucket, at most kLsSubMax sub-buckets
+            int sb = 0;
+            while (sb < 10 && (m >> (sb + 3)) > 0) ++sb;
+            if (sb > shift) sb = shift;
+            const int ssh = shift - sb;
+            const unsigned int ns = 1u << sb, smask = ns - 1u;
+            for (unsigned int i = threadIdx.x; i < ns; i += kBkThreads) S.sub[i] = 0;
             __syncthreads();
-            unsigned int before = 0;
-            for (int w = 0; w < warp; ++w) before += S.wsum[w];
-            unsigned int run = before + x - t;
+            for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
+                const unsigned long long kk = k[lo + i];
+                S.k1[i] = kk;
+                S.v1[i] = v[lo + i];
+                atomicAdd(&S.sub[(unsigned int)(kk >> ssh) & smask], 1u);
+            }
+            __syncthreads();
+            {   // exclusive scan of ns (<= 1024) sub-bucket counts: 4 per thread
+                unsigned int c[4], t = 0;
 #pragma unroll
-            for (int q = 0; q < 4; ++q) {
-                const unsigned int i = threadIdx.x * 4 + q;
-                if (i < ns) { S.sub[i] = run; S.cur[i] = run; }
-                run += c[q];
+                for (int q = 0; q < 4; ++q) {
+                    const unsigned int i = threadIdx.x * 4 + q;
+                    c[q] = i < ns ? S.sub[i] : 0u;
+                    t += c[q];
+                }
+                unsigned int x = t;
+#pragma unroll
+                for (int o = 1; o < 32; o <<= 1) {
+                    const unsigned int y = __shfl_up_sync(kFull, x, o);
+                    if (lane >= o) x += y;
+                }
+                if (lane == 31) S.wsum[warp] = x;
+                __syncthreads();
+                unsigned int before = 0;
+                for (int w = 0; w < warp; ++w) before += S.wsum[w];
+                unsigned int run = before + x - t;
+#pragma unroll
+                for (int q = 0; q < 4; ++q) {
+                    const unsigned int i = threadIdx.x * 4 + q;
+                    if (i < ns) { S.sub[i] = run; S.cur[i] = run; }
+                    run += c[q];
+                }
+                if (threadIdx.x == kBkThreads - 1) S.sub[ns] = run;
             }
-            if (threadIdx.x == kBkThreads - 1) S.sub[ns] = run;
+            __syncthreads();
+            for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
+                const unsigned long long kk = S.k1[i];
+                const unsigned int p = atomicAdd(&S.cur[(unsigned int)(kk >> ssh) & smask], 1u);
+                S.k2[p] = kk;
+                S.v2[p] = S.v1[i];
+            }
+            __syncthreads();
+            for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {  // rank -> sorted smem
+                const unsigned long long kk = S.k2[i];
+                const unsigned int sbk = (unsigned int)(kk >> ssh) & smask;
+                const unsigned int s0 = S.sub[sbk], s1 = S.sub[sbk + 1];
+                unsigned int rank = s0;
+                for (unsigned int j = s0; j < s1; ++j) {
+                    const unsigned long long kj = S.k2[j];
+                    rank += (kj < kk) | ((kj == kk) & (j < i));
+                }
+                S.k1[rank] = kk;
+                S.v1[rank] = S.v2[i];
+            }
+            __syncthreads();
+            if (tiefix) {  // runs of equal 64-bit prefixes never cross buckets
+                for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
+                    const unsigned long long ki = S.k1[i];
+                    if (i > 0 && S.k1[i - 1] == ki) continue;          // not a run head
+                    if (i + 1 >= m || S.k1[i + 1] != ki) continue;     // run of one
+                    unsigned int j = i + 1;
+                    while (j < m && S.k1[j] == ki && j - i <= (unsigned)kMaxRun) ++j;
+                    if (j - i > (unsigned)kMaxRun) { atomicOr(flag, 1u); continue; }
+                    for (unsigned int t = i + 1; t < j; ++t) {  // insertion sort by the full tuple
+                        const unsigned int x = S.v1[t];
+                        const Q18Row rx = rows[x];
+                        const long long ax = amt[x];
+                        int u = (int)t - 1;
+                        while (u >= (int)i && row_less(rx, ax, rows[S.v1[u]], amt[S.v1[u]])) {
+                            S.v1[u + 1] = S.v1[u];
+                            --u;
+                        }
+                        S.v1[u + 1] = x;
+                    }
+                }
+                __syncthreads();
+            }
         }
         __syncthreads();
-        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
-            const unsigned long long kk = S.k1[i];
-            const unsigned int p = atomicAdd(&S.cur[(unsigned int)(kk >> ssh) & smask], 1u);
-            S.k2[p] = kk;
-            S.v2[p] = S.v1[i];
-        }
-        __syncthreads();
-        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
-            const unsigned long long kk = S.k2[i];
-            const unsigned int sbk = (unsigned int)(kk >> ssh) & smask;
-            const unsigned int s0 = S.sub[sbk], s1 = S.sub[sbk + 1];
-            unsigned int rank = s0;
-            for (unsigned int j = s0; j < s1; ++j) {
-                const unsigned long long kj = S.k2[j];
-                rank += (kj < kk) | ((kj == kk) & (j < i));
+        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {  // emit at final positions
+            const unsigned int r = S.v1[i];
+            Q18Row row;
+            {
+                unsigned long long *w64 = reinterpret_cast<unsigned long long *>(&row);
+                ld16_policy(rows + r, w64[0], w64[1], drop);
+                ld16_policy(reinterpret_cast<const char *>(rows + r) + 16, w64[2], w64[3], drop);
             }
-            k[lo + rank] = kk;
-            v[lo + rank] = S.v2[i];
+            const unsigned long long a = sp.bits_a ? (S.k1[i] >> ashift) : 0ull;
+            const uint64_t j = lo + i;
+            dst.c_last[j] = row.c_last;
+            dst.c_id[j] = row.c_id;
+            dst.o_id[j] = row.o_id;
+            dst.o_entry_d[j] = row.o_entry_d;
+            dst.o_ol_cnt[j] = row.o_ol_cnt;
+            dst.amount_sum[j] = m == 1 && plan->n <= 1 ? amt[r]
+                                                       : (long long)((unsigned long long)sp.amt_max - a);
+            dst.o_w_id[j] = row.o_w_id;
+            dst.o_d_id[j] = row.o_d_id;
         }
         __syncthreads();
     }
@@ -619,20 +619,20 @@ bucket_local_sort_kernel(unsigned long long *__restrict__ k, unsigned int *__res
 
 }  // namespace
 
-void bucket_sort_pairs(uint64_t n_max, const unsigned long long *dn, const int *dshift,
-                       int bucket_bits, const BucketSort &s, unsigned int *flag, int num_sms,
-                       cudaStream_t st, PhaseMarks *marks) {
+void q18_bucket_order(const Q18Row *rows, const long long *amt, const Q18Plan *plan, uint64_t n_max,
+                      int bucket_bits, const BucketSort &s, const Q18Cols &dst, unsigned int *flag,
+                      int num_sms, cudaStream_t st, PhaseMarks *marks) {
     auto begin = [&](const char *nm) { if (marks) marks->begin(nm); };
     auto end = [&] { if (marks) marks->end(); };
     if (bucket_bits > kBucketMaxBits) bucket_bits = kBucketMaxBits;
     const int nb = 1 << bucket_bits;
     static bool init = false;
     if (!init) {
-        cudaFuncSetAttribute(bucket_local_sort_kernel<kLsCapSmall, 0>,
+        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapSmall, 0>,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapSmall>));
-        cudaFuncSetAttribute(bucket_local_sort_kernel<kLsCapLarge, kLsCapSmall>,
+        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall>,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapLarge>));
-        cudaFuncSetAttribute(bucket_hist_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+        cudaFuncSetAttribute(q18_keys_hist_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
                              4 << kBucketMaxBits);
         cudaFuncSetAttribute(bucket_scatter_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
                              4 << kBucketMaxBits);
@@ -640,35 +640,32 @@ void bucket_sort_pairs(uint64_t n_max, const unsigned long long *dn, const int *
     }
     cudaMemsetAsync(s.count, 0, sizeof(unsigned int) * (nb + 1), st);
     cudaMemsetAsync(s.big, 0, sizeof(unsigned int), st);
-    const uint64_t per = (uint64_t)kBkThreads * kBkItems;
-    uint64_t hb = (n_max + per - 1) / per;
-    if (hb > (uint64_t)num_sms * 2) hb = (uint64_t)num_sms * 2;
-    if (!hb) hb = 1;
-    begin("q18_bucket_hist");
-    bucket_hist_kernel<<<(unsigned)hb, kBkThreads, nb * 4, st>>>(s.k[0], dn, dshift, nb, s.count);
-    count_launches(1);
-    end();
-    begin("q18_bucket_scan");
-    bucket_scan_kernel<<<1, 1024, 0, st>>>(s.count, nb, s.offset, s.cursor);
+    const uint64_t n1 = n_max ? n_max : 1;
+    uint64_t hb = (n1 + kBkThreads * 8 - 1) / (kBkThreads * 8);
+    if (hb > (uint64_t)num_sms * 4) hb = (uint64_t)num_sms * 4;
+    begin("q18_sort_keys_hist");
+    q18_keys_hist_kernel<<<(unsigned)hb, kBkThreads, nb * 4, st>>>(rows, amt, plan, s.k[0], s.v[0], nb,
+                                                                  s.count, s.offset, s.cursor, s.ticket);
     count_launches(1);
     end();
     begin("q18_bucket_scatter");
-    const uint64_t sb = (n_max + per - 1) / per;
-    bucket_scatter_kernel<<<(unsigned)(sb ? sb : 1), kBkThreads, nb * 4, st>>>(
-        s.k[0], s.v[0], s.k[1], s.v[1], dn, dshift, nb, s.cursor);
+    const uint64_t per = (uint64_t)kBkThreads * kBkItems;
+    const uint64_t sb = (n1 + per - 1) / per;
+    bucket_scatter_kernel<<<(unsigned)sb, kBkThreads, nb * 4, st>>>(s.k[0], s.v[0], s.k[1], s.v[1], plan,
+                                                                   nb, s.cursor);
     count_launches(1);
     end();
-    begin("q18_bucket_local");
+    begin("q18_bucket_sort_emit");
     unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
-    bucket_local_sort_kernel<kLsCapSmall, 0><<<lb, kBkThreads, sizeof(LsSmem<kLsCapSmall>), st>>>(
-        s.k[1], s.v[1], s.offset, nb, dshift, flag, s.big);
+    bucket_local_emit_kernel<kLsCapSmall, 0><<<lb, kBkThreads, sizeof(LsSmem<kLsCapSmall>), st>>>(
+        s.k[1], s.v[1], s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
     end();
     // buckets above the small capacity (skewed keys): one block per SM, ~200 KB shared memory
-    begin("q18_bucket_local_large");
-    bucket_local_sort_kernel<kLsCapLarge, kLsCapSmall><<<(unsigned)num_sms, kBkThreads,
+    begin("q18_bucket_sort_emit_large");
+    bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall><<<(unsigned)num_sms, kBkThreads,
                                                           sizeof(LsSmem<kLsCapLarge>), st>>>(
-        s.k[1], s.v[1], s.offset, nb, dshift, flag, s.big);
+        s.k[1], s.v[1], s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
     end();
 }

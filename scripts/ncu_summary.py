@@ -59,11 +59,9 @@ if traffic:
     marks = {"q6_kernel": "q6_scan_filter_sum", "q1_kernel": "q1_scan_filter_groupby",
              "q18_init_kernel": "q18_init", "q18_build_kernel": "q18_build",
              "q18_probe_kernel": "q18_probe_groupjoin", "q18_having_kernel": "q18_having_compact",
-             "sort_keys_kernel": "q18_sort_keys", "tiefix_kernel": "q18_tiefix",
-             "permute_kernel": "q18_permute", "bucket_hist_kernel": "q18_bucket_hist",
-             "bucket_scan_kernel": "q18_bucket_scan", "bucket_scatter_kernel": "q18_bucket_scatter",
-             "bucket_local_sort_kernel<2048, 0>": "q18_bucket_local",
-             "bucket_local_sort_kernel<8192, 2048>": "q18_bucket_local_large",
+             "q18_keys_hist_kernel": "q18_sort_keys_hist", "bucket_scatter_kernel": "q18_bucket_scatter",
+             "bucket_local_emit_kernel<2048, 0>": "q18_bucket_sort_emit",
+             "bucket_local_emit_kernel<8192, 2048>": "q18_bucket_sort_emit_large",
              "q18_plan_kernel": "q18_plan", "q1_compact_kernel": "q1_compact",
              "q1_emit_kernel": "q1_emit"}
     bymark = {}
