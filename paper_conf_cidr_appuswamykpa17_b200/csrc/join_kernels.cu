@@ -96,14 +96,13 @@ __device__ __forceinline__ void jx_clear(const JoinIndex &j, uint64_t i) {
     else reinterpret_cast<ulonglong2 *>(j.ht)[i] = make_ulonglong2(kEmpty, 0ull);
 }
 
-__global__ void q18_init_kernel(Q18Scratch s, uint64_t n_orders) {
+__global__ void q18_init_kernel(Q18Scratch s) {
     const uint64_t a = jx_words(s.jo), b = jx_words(s.jc);
-    const uint64_t total = a + b + n_orders;
+    const uint64_t total = a + b;  // (the accumulators are zeroed by the build, row by row)
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < total; i += stride) {
         if (i < a) jx_clear(s.jo, i);
-        else if (i < a + b) jx_clear(s.jc, i - a);
-        else reinterpret_cast<ulonglong2 *>(s.acc)[i - a - b] = make_ulonglong2(0ull, 0ull);
+        else jx_clear(s.jc, i - a);
     }
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         *s.err = 0;
@@ -125,6 +124,7 @@ __global__ void q18_build_kernel(const int32_t *__restrict__ o_w, const int32_t 
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n_o + n_c; i += stride) {
         bool ok;
         if (i < n_o) {
+            reinterpret_cast<ulonglong2 *>(s.acc)[i] = make_ulonglong2(0ull, 0ull);  // acc[orders row]
             ok = jx_insert(s.jo, o_w[i], o_d[i], o_id[i], (unsigned int)i, s.err, kErrDupOrders);
         } else {
             const uint64_t j = i - n_o;
@@ -422,8 +422,9 @@ __global__ void q18_stats_kernel(const Q18Row *__restrict__ rows, const long lon
 }  // namespace
 
 void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st) {
-    const uint64_t words = jx_words(s.jo) + jx_words(s.jc) + n_orders;
-    q18_init_kernel<<<grid_for(words, 256, num_sms, 8), 256, 0, st>>>(s, n_orders);
+    (void)n_orders;
+    const uint64_t words = jx_words(s.jo) + jx_words(s.jc);
+    q18_init_kernel<<<grid_for(words, 256, num_sms, 8), 256, 0, st>>>(s);
     count_launches(1);
 }
 
