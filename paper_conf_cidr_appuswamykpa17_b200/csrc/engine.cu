@@ -15,6 +15,7 @@
 #include <chrono>
 #include <cstdarg>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <deque>
 #include <map>
@@ -280,6 +281,10 @@ struct Prof {  // per-kernel CUDA events on the compute stream
 // ============================================================= engine ===
 struct h2tap_engine {
     int device = 0, rank = 0, world = 1, num_sms = 148;
+    // Q6/Q1 stream their columns with TMA bulk copies (H2TAP_SCAN=ldg: register-prefetch kernels);
+    // the Q18 probe keeps register prefetch at high occupancy — its dependent lookups and atomics
+    // need more warps than a one-block-per-SM shared-memory ring leaves (H2TAP_PROBE=tma: ring)
+    bool scan_tma = true, probe_tma = false;
     ncclComm_t comm = nullptr;
     cudaStream_t compute = nullptr, copy = nullptr;
     cudaEvent_t q_begin = nullptr, q_end = nullptr;
@@ -609,9 +614,10 @@ void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.done_counter = static_cast<unsigned int *>(e->arena.get("q6.counter", 64, true, e->compute));
     s.out = static_cast<long long *>(e->arena.get("q6.out", 64));
     e->prof.run("q6_scan_filter_sum", [&] {
-        launch_q6(colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D), colp<int32_t>(v, T, H2TAP_OL_QUANTITY),
-                  colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T], q.p[0], q.p[1], q.p[2], q.p[3], s,
-                  e->num_sms, e->compute);
+        (e->scan_tma ? launch_q6_tma : launch_q6)(
+            colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D), colp<int32_t>(v, T, H2TAP_OL_QUANTITY),
+            colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T], q.p[0], q.p[1], q.p[2], q.p[3], s,
+            e->num_sms, e->compute);
         CK(cudaGetLastError());
     });
     if (e->world > 1)
@@ -658,7 +664,7 @@ void launch_q1_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.o_cnt = static_cast<long long *>(dev_block(e, q, 8 * kQ1MaxGroups));
     if (fresh) launch_q1_reset(s, e->compute);  // tables self-clean afterwards (q1_compact)
     e->prof.run("q1_scan_filter_groupby", [&] {
-        launch_q1(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
+        (e->scan_tma ? launch_q1_tma : launch_q1)(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
                   colp<int32_t>(v, T, H2TAP_OL_QUANTITY), colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T],
                   q.p[0], s, e->num_sms, e->compute);
         CK(cudaGetLastError());
@@ -844,7 +850,7 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     });
     e->prof.run("q18_probe_groupjoin", [&] {
         if (n_ol)
-            launch_q18_probe(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
+            (e->probe_tma ? launch_q18_probe_tma : launch_q18_probe)(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
                              colp<int32_t>(v, OL, H2TAP_OL_O_ID), colp<int64_t>(v, OL, H2TAP_OL_AMOUNT),
                              n_ol, s, e->num_sms, e->compute);
     });
@@ -1145,6 +1151,8 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
             return fail(H2TAP_ECUDA, "built for sm_100a (B200); device %d is sm_%d%d", e->device,
                         prop.major, prop.minor);
         e->num_sms = prop.multiProcessorCount;
+        if (const char *impl = std::getenv("H2TAP_SCAN")) e->scan_tma = std::strcmp(impl, "ldg") != 0;
+        if (const char *impl = std::getenv("H2TAP_PROBE")) e->probe_tma = std::strcmp(impl, "tma") == 0;
 
         CK(cudaStreamCreateWithFlags(&e->compute, cudaStreamNonBlocking));
         CK(cudaStreamCreateWithFlags(&e->copy, cudaStreamNonBlocking));

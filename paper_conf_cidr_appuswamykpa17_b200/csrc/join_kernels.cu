@@ -14,6 +14,7 @@
 #include <cstdint>
 #include <cuda_runtime.h>
 
+#include "bulk_pipeline.cuh"
 #include "cache_hints.cuh"
 #include "kernels.cuh"
 
@@ -156,6 +157,47 @@ __device__ __forceinline__ void flush_run(const Q18Scratch &s, const Key3 &k, lo
     }
 }
 
+// One warp step over 128 consecutive rows, 4 per lane (k, a in registers; `valid` per lane):
+// in-lane runs, cross-lane segmented scan, one probe + two atomics per run (see above).
+__device__ __forceinline__ void probe_lane_group(const Q18Scratch &s, const Key3 (&k)[4],
+                                                 const long long (&a)[4], bool valid, int lane) {
+        // in-lane runs: b[j] = row j starts a run; s[j], c[j] = running sum / count of its run
+        bool b1 = !eq3(k[1], k[0]), b2 = !eq3(k[2], k[1]), b3 = !eq3(k[3], k[2]);
+        long long s0 = a[0], s1 = (b1 ? 0 : s0) + a[1], s2 = (b2 ? 0 : s1) + a[2], s3 = (b3 ? 0 : s2) + a[3];
+        unsigned c0 = 1, c1 = (b1 ? 0 : c0) + 1, c2 = (b2 ? 0 : c1) + 1, c3 = (b3 ? 0 : c2) + 1;
+        const bool multi = b1 | b2 | b3;
+        // does my first run continue the previous lane's last run?
+        const int pw = __shfl_up_sync(kFull, k[3].w, 1), pd = __shfl_up_sync(kFull, k[3].d, 1),
+                  po = __shfl_up_sync(kFull, k[3].o, 1);
+        const bool pvalid = __shfl_up_sync(kFull, valid, 1);
+        const bool cont = lane > 0 && valid && pvalid && pw == k[0].w && pd == k[0].d && po == k[0].o;
+        const bool next_cont = __shfl_down_sync(kFull, cont, 1) && lane < 31;
+        // segmented inclusive scan of the lanes' last partial runs (segment starts where a lane
+        // does not continue, or where its last run starts inside the lane)
+        const bool start = !cont || multi;
+        const unsigned starts = __ballot_sync(kFull, start);
+        const int seg = 31 - __clz(starts & (0xffffffffu >> (31 - lane)));
+        long long is = s3;
+        unsigned ic = c3;
+#pragma unroll
+        for (int off = 1; off < 32; off <<= 1) {
+            const long long ts = __shfl_up_sync(kFull, is, off);
+            const unsigned tc = __shfl_up_sync(kFull, ic, off);
+            if (lane - off >= seg) { is += ts; ic += tc; }
+        }
+        // carry into my first run = inclusive value of the previous lane (if I continue it)
+        long long carry_s = __shfl_up_sync(kFull, is, 1);
+        unsigned carry_c = __shfl_up_sync(kFull, ic, 1);
+        if (!cont) { carry_s = 0; carry_c = 0; }
+        if (!valid) return;
+        // runs ending inside the lane (rows 0..2): the first run also gets the carry
+        if (b1) flush_run(s, k[0], s0 + carry_s, c0 + carry_c);
+        if (b2) flush_run(s, k[1], s1 + (b1 ? 0 : carry_s), c1 + (b1 ? 0 : carry_c));
+        if (b3) flush_run(s, k[2], s2 + ((b1 | b2) ? 0 : carry_s), c2 + ((b1 | b2) ? 0 : carry_c));
+        // the lane's last run ends here unless the next lane continues it
+        if (!next_cont) flush_run(s, k[3], is, ic);
+}
+
 __global__ void __launch_bounds__(kProbeThreads)
 q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ ol_d,
                  const int32_t *__restrict__ ol_o, const int64_t *__restrict__ ol_amt, uint64_t n,
@@ -193,46 +235,91 @@ q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ o
         } else {
             for (int j = 0; j < 4; ++j) { k[j] = {0, 0, 0}; a[j] = 0; }
         }
-        // in-lane runs: b[j] = row j starts a run; s[j], c[j] = running sum / count of its run
-        bool b1 = !eq3(k[1], k[0]), b2 = !eq3(k[2], k[1]), b3 = !eq3(k[3], k[2]);
-        long long s0 = a[0], s1 = (b1 ? 0 : s0) + a[1], s2 = (b2 ? 0 : s1) + a[2], s3 = (b3 ? 0 : s2) + a[3];
-        unsigned c0 = 1, c1 = (b1 ? 0 : c0) + 1, c2 = (b2 ? 0 : c1) + 1, c3 = (b3 ? 0 : c2) + 1;
-        const bool multi = b1 | b2 | b3;
-        // does my first run continue the previous lane's last run?
-        const int pw = __shfl_up_sync(kFull, k[3].w, 1), pd = __shfl_up_sync(kFull, k[3].d, 1),
-                  po = __shfl_up_sync(kFull, k[3].o, 1);
-        const bool pvalid = __shfl_up_sync(kFull, valid, 1);
-        const bool cont = lane > 0 && valid && pvalid && pw == k[0].w && pd == k[0].d && po == k[0].o;
-        const bool next_cont = __shfl_down_sync(kFull, cont, 1) && lane < 31;
-        // segmented inclusive scan of the lanes' last partial runs (segment starts where a lane
-        // does not continue, or where its last run starts inside the lane)
-        const bool start = !cont || multi;
-        const unsigned starts = __ballot_sync(kFull, start);
-        const int seg = 31 - __clz(starts & (0xffffffffu >> (31 - lane)));
-        long long is = s3;
-        unsigned ic = c3;
-#pragma unroll
-        for (int off = 1; off < 32; off <<= 1) {
-            const long long ts = __shfl_up_sync(kFull, is, off);
-            const unsigned tc = __shfl_up_sync(kFull, ic, off);
-            if (lane - off >= seg) { is += ts; ic += tc; }
-        }
-        // carry into my first run = inclusive value of the previous lane (if I continue it)
-        long long carry_s = __shfl_up_sync(kFull, is, 1);
-        unsigned carry_c = __shfl_up_sync(kFull, ic, 1);
-        if (!cont) { carry_s = 0; carry_c = 0; }
-        if (!valid) continue;
-        // runs ending inside the lane (rows 0..2): the first run also gets the carry
-        if (b1) flush_run(s, k[0], s0 + carry_s, c0 + carry_c);
-        if (b2) flush_run(s, k[1], s1 + (b1 ? 0 : carry_s), c1 + (b1 ? 0 : carry_c));
-        if (b3) flush_run(s, k[2], s2 + ((b1 | b2) ? 0 : carry_s), c2 + ((b1 | b2) ? 0 : carry_c));
-        // the lane's last run ends here unless the next lane continues it
-        if (!next_cont) flush_run(s, k[3], is, ic);
+        probe_lane_group(s, k, a, valid, lane);
     }
     // ragged tail (< 4 rows) plus nothing else: one thread, row at a time
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         for (uint64_t i = nvec * 4; i < n; ++i)
             flush_run(s, Key3{ol_w[i], ol_d[i], ol_o[i]}, ol_amt[i], 1u);
+    }
+}
+
+// K4, TMA-bulk pipelined variant: one block per SM, the last warp streams 3072-row chunks of
+// w, d, o and amount into a 3-stage ring (180 KB); each of the 24 consumer warps runs
+// probe_lane_group on 128 rows of the chunk straight from shared memory (128-bit shared loads).
+constexpr int kProbeTmaWarps = 24;                 // the lookups and atomics need warps in flight
+constexpr int kProbeChunk = kProbeTmaWarps * 128;  // 128 rows per consumer warp per chunk
+constexpr int kProbeStages = 3;                    // 3 x 60 KB
+struct ProbeStages {
+    long long amt[kProbeStages][kProbeChunk];
+    int w[kProbeStages][kProbeChunk], d[kProbeStages][kProbeChunk], o[kProbeStages][kProbeChunk];
+    uint64_t full[kProbeStages], empty[kProbeStages];
+};
+
+__global__ void __launch_bounds__((kProbeTmaWarps + 1) * 32, 1)
+q18_probe_tma_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ ol_d,
+                     const int32_t *__restrict__ ol_o, const int64_t *__restrict__ ol_amt, uint64_t n,
+                     Q18Scratch s) {
+    extern __shared__ __align__(128) unsigned char smem_raw[];
+    ProbeStages &P = *reinterpret_cast<ProbeStages *>(smem_raw);
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    if (threadIdx.x == 0) {
+        for (int st = 0; st < kProbeStages; ++st) {
+            mbar_init(&P.full[st], 1);
+            mbar_init(&P.empty[st], kProbeTmaWarps);
+        }
+        fence_mbar_init();
+    }
+    __syncthreads();
+    const uint64_t nchunks = (n + kProbeChunk - 1) / kProbeChunk;
+    if (warp == kProbeTmaWarps) {  // producer
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            int it = 0;
+            for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
+                const int st = it % kProbeStages;
+                const unsigned ph = (unsigned)(it / kProbeStages) & 1u;
+                if (it >= kProbeStages) mbar_wait(&P.empty[st], ph ^ 1u);
+                const uint64_t r0 = c * kProbeChunk;
+                const unsigned rows = (unsigned)(n - r0 < (uint64_t)kProbeChunk ? n - r0 : (uint64_t)kProbeChunk);
+                const unsigned b8 = round16(rows * 8), b4 = round16(rows * 4);
+                mbar_arrive_expect_tx(&P.full[st], b8 + 3 * b4);
+                bulk_g2s(P.amt[st], ol_amt + r0, b8, &P.full[st], pol);
+                bulk_g2s(P.w[st], ol_w + r0, b4, &P.full[st], pol);
+                bulk_g2s(P.d[st], ol_d + r0, b4, &P.full[st], pol);
+                bulk_g2s(P.o[st], ol_o + r0, b4, &P.full[st], pol);
+            }
+        }
+        return;
+    }
+    int it = 0;
+    for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
+        const int st = it % kProbeStages;
+        mbar_wait(&P.full[st], (unsigned)(it / kProbeStages) & 1u);
+        const unsigned rows = (unsigned)(n - c * kProbeChunk < (uint64_t)kProbeChunk ? n - c * kProbeChunk
+                                                                                    : (uint64_t)kProbeChunk);
+        const unsigned r = warp * 128 + lane * 4;  // this lane's 4 consecutive rows
+        Key3 k[4];
+        long long a[4];
+        const bool valid = r + 3 < rows;
+        if (valid) {
+            const int4 W = *reinterpret_cast<const int4 *>(&P.w[st][r]);
+            const int4 D = *reinterpret_cast<const int4 *>(&P.d[st][r]);
+            const int4 O = *reinterpret_cast<const int4 *>(&P.o[st][r]);
+            const longlong2 A0 = *reinterpret_cast<const longlong2 *>(&P.amt[st][r]);
+            const longlong2 A1 = *reinterpret_cast<const longlong2 *>(&P.amt[st][r + 2]);
+            k[0] = {W.x, D.x, O.x}; k[1] = {W.y, D.y, O.y}; k[2] = {W.z, D.z, O.z}; k[3] = {W.w, D.w, O.w};
+            a[0] = A0.x; a[1] = A0.y; a[2] = A1.x; a[3] = A1.y;
+        } else {
+            for (int j = 0; j < 4; ++j) { k[j] = {0, 0, 0}; a[j] = 0; }
+        }
+        // rows of a partial last group (< 4, last chunk only) go one by one, straight from smem
+        if (!valid && r < rows)
+            for (unsigned j = r; j < rows; ++j)
+                flush_run(s, Key3{P.w[st][j], P.d[st][j], P.o[st][j]}, P.amt[st][j], 1u);
+        __syncwarp();
+        if (lane == 0) mbar_arrive(&P.empty[st]);  // registers hold everything from here on
+        probe_lane_group(s, k, a, valid, lane);
     }
 }
 
@@ -441,6 +528,22 @@ void launch_q18_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *o
                       cudaStream_t st) {
     q18_probe_kernel<<<grid_for((n_ol + 3) / 4, kProbeThreads, num_sms, 8), kProbeThreads, 0, st>>>(
         ol_w, ol_d, ol_o, ol_amt, n_ol, s);
+    count_launches(1);
+}
+
+void launch_q18_probe_tma(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
+                          const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
+                          cudaStream_t st) {
+    static bool init = false;
+    if (!init) {
+        cudaFuncSetAttribute(q18_probe_tma_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             (int)sizeof(ProbeStages));
+        init = true;
+    }
+    const uint64_t nchunks = (n_ol + kProbeChunk - 1) / kProbeChunk;
+    const unsigned grid = (unsigned)(nchunks < (uint64_t)num_sms ? (nchunks ? nchunks : 1) : num_sms);
+    q18_probe_tma_kernel<<<grid, (kProbeTmaWarps + 1) * 32, sizeof(ProbeStages), st>>>(ol_w, ol_d, ol_o,
+                                                                                      ol_amt, n_ol, s);
     count_launches(1);
 }
 

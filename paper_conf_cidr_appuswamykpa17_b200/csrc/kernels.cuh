@@ -21,6 +21,10 @@ int q6_max_blocks(int num_sms);
 void launch_q6(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uint64_t n,
                int64_t d_lo, int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s,
                int num_sms, cudaStream_t st);
+// same result, TMA-bulk (cp.async.bulk) staged through a shared-memory ring, one block per SM
+void launch_q6_tma(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uint64_t n,
+                   int64_t d_lo, int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s,
+                   int num_sms, cudaStream_t st);
 
 // ----------------------------------------------------------------- Q1 (K2) --
 // GROUP BY ol_number over rows with delivery > cutoff; per group (count, sum_qty, sum_amount).
@@ -43,6 +47,9 @@ void launch_q1_reset(const Q1Scratch &s, cudaStream_t st);
 void launch_q1(const int32_t *number, const int64_t *deliv, const int32_t *qty,
                const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int num_sms,
                cudaStream_t st);
+void launch_q1_tma(const int32_t *number, const int64_t *deliv, const int32_t *qty,
+                   const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int num_sms,
+                   cudaStream_t st);  // same result, TMA-bulk staged, one block per SM
 void launch_q1_compact(const Q1Scratch &s, cudaStream_t st);        // tables -> groups[], ngroups
 void launch_q1_merge(const Q1Group *all, uint64_t n, const Q1Scratch &s, cudaStream_t st);
 void launch_q1_emit(const Q1Scratch &s, uint64_t max_groups, cudaStream_t st);  // rank by key + AVG;
@@ -99,6 +106,9 @@ void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_i
 void launch_q18_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
                       const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
                       cudaStream_t st);
+void launch_q18_probe_tma(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
+                          const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
+                          cudaStream_t st);  // same result, TMA-bulk staged, one block per SM
 void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id,
                        const int32_t *o_c, const int32_t *o_cnt, const int64_t *o_ent,
                        uint64_t n_o, const int32_t *c_last, int64_t having,

@@ -7,9 +7,11 @@
 // one CUDA kernel per primitive with materialised intermediates and calls that sub-optimal
 // (L527-535) with fusion as future work (L552-554): here each query is ONE fused kernel plus a
 // tiny finaliser, and the scan is HBM-bound (20 B/row for Q6, 24 B/row for Q1).
+#include <algorithm>
 #include <cstdint>
 #include <cuda_runtime.h>
 
+#include "bulk_pipeline.cuh"
 #include "kernels.cuh"
 
 namespace h2tap {
@@ -148,6 +150,107 @@ q6_kernel(const longlong2 *__restrict__ deliv, const int4 *__restrict__ qty,
     }
 }
 
+// ------------------------------------------------- Q6, TMA-bulk pipelined variant --
+// One persistent block per SM: warp 8's elected lane streams 2048-row chunks of the three columns
+// into a 4-stage shared-memory ring with cp.async.bulk (mbarrier complete_tx); warps 0-7
+// evaluate the predicate from shared memory and release the stage. 160 KB in flight per SM
+// without any load registers; same arithmetic and last-block fold as q6_kernel.
+constexpr int kTmaConsumerWarps = 8;
+constexpr int kTmaThreads = (kTmaConsumerWarps + 1) * 32;
+constexpr int kQ6Chunk = 2048;
+constexpr int kQ6Stages = 4;
+struct Q6TmaSmem {
+    long long deliv[kQ6Stages][kQ6Chunk];
+    long long amt[kQ6Stages][kQ6Chunk];
+    int qty[kQ6Stages][kQ6Chunk];
+    uint64_t full[kQ6Stages], empty[kQ6Stages];
+};
+
+__global__ void __launch_bounds__(kTmaThreads, 1)
+q6_tma_kernel(const long long *__restrict__ deliv, const int *__restrict__ qty,
+              const long long *__restrict__ amt, uint64_t n, Q6Pred pred,
+              long long *__restrict__ part, unsigned int *__restrict__ counter,
+              long long *__restrict__ out) {
+    extern __shared__ __align__(128) unsigned char smem_raw[];
+    Q6TmaSmem &S = *reinterpret_cast<Q6TmaSmem *>(smem_raw);
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const uint64_t nchunks = (n + kQ6Chunk - 1) / kQ6Chunk;
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < kQ6Stages; ++s) {
+            mbar_init(&S.full[s], 1);
+            mbar_init(&S.empty[s], kTmaConsumerWarps);
+        }
+        fence_mbar_init();
+    }
+    __syncthreads();
+    long long sum = 0, cnt = 0;
+    if (warp == kTmaConsumerWarps) {  // producer
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            int it = 0;
+            for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
+                const int s = it % kQ6Stages;
+                const unsigned ph = (unsigned)(it / kQ6Stages) & 1u;
+                if (it >= kQ6Stages) mbar_wait(&S.empty[s], ph ^ 1u);
+                const uint64_t r0 = c * kQ6Chunk;
+                const unsigned rows = (unsigned)(n - r0 < (uint64_t)kQ6Chunk ? n - r0 : (uint64_t)kQ6Chunk);
+                const unsigned b8 = round16(rows * 8), b4 = round16(rows * 4);
+                mbar_arrive_expect_tx(&S.full[s], 2 * b8 + b4);
+                bulk_g2s(S.deliv[s], deliv + r0, b8, &S.full[s], pol);
+                bulk_g2s(S.amt[s], amt + r0, b8, &S.full[s], pol);
+                bulk_g2s(S.qty[s], qty + r0, b4, &S.full[s], pol);
+            }
+        }
+    } else {  // consumers
+        int it = 0;
+        for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
+            const int s = it % kQ6Stages;
+            mbar_wait(&S.full[s], (unsigned)(it / kQ6Stages) & 1u);
+            const unsigned rows = (unsigned)(n - c * kQ6Chunk < (uint64_t)kQ6Chunk ? n - c * kQ6Chunk : (uint64_t)kQ6Chunk);
+#pragma unroll 4
+            for (unsigned r = threadIdx.x; r < rows; r += kTmaConsumerWarps * 32) {
+                const long long d = S.deliv[s][r];
+                const bool p = pred(d, S.qty[s][r]);
+                sum += p ? S.amt[s][r] : 0;
+                cnt += p;
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&S.empty[s]);
+        }
+    }
+    // block reduction (9 warps) -> per-block partial -> last block folds all partials
+    __shared__ long long s_sum[kTmaConsumerWarps + 1], s_cnt[kTmaConsumerWarps + 1];
+    __shared__ bool s_last;
+    sum = warp_sum(sum);
+    cnt = warp_sum(cnt);
+    if (lane == 0) { s_sum[warp] = sum; s_cnt[warp] = cnt; }
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        long long S0 = 0, C0 = 0;
+        for (int w = 0; w <= kTmaConsumerWarps; ++w) { S0 += s_sum[w]; C0 += s_cnt[w]; }
+        part[2 * blockIdx.x] = S0;
+        part[2 * blockIdx.x + 1] = C0;
+        __threadfence();
+        s_last = atomicAdd(counter, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (s_last && warp == 0) {
+        __threadfence();
+        long long ts = 0, tc = 0;
+        for (unsigned b = lane; b < gridDim.x; b += 32) {
+            ts += __ldcg(part + 2 * b);
+            tc += __ldcg(part + 2 * b + 1);
+        }
+        ts = warp_sum(ts);
+        tc = warp_sum(tc);
+        if (lane == 0) {
+            out[0] = ts;
+            out[1] = tc;
+            *counter = 0;
+        }
+    }
+}
+
 // ================================================================== Q1 ====
 constexpr int kQ1Threads = 256;
 constexpr int kQ1Unroll = 2;   // 4-row vectors per lane per warp iteration
@@ -217,6 +320,26 @@ __device__ __forceinline__ void q1_sparse_warp(Q1Smem &sm, const Q1Scratch &g, b
         need = need && !in;
         pend &= ~grp;
     }
+}
+
+// Block end: dense keys, one warp per key, one global atomic per (key, accumulator) per block;
+// the block's sparse table into the global table. Threads tid < kQ1Threads take part.
+__device__ void q1_block_merge(Q1Smem &sm, const Q1Scratch &g, int tid) {
+    if (tid >= kQ1Threads) return;
+    const int lane = tid & 31, warp = tid >> 5;
+    for (int k = warp; k < kQ1Dense; k += kQ1Threads / 32) {
+        long long c = 0, q = 0, a = 0;
+        for (int t = lane; t < kQ1Threads; t += 32) { c += sm.cnt[k][t]; q += sm.qty[k][t]; a += sm.amt[k][t]; }
+        c = warp_sum(c); q = warp_sum(q); a = warp_sum(a);
+        if (lane == 0 && c) {
+            atomicAdd(g.dense + 3 * k + 0, (unsigned long long)c);
+            atomicAdd(g.dense + 3 * k + 1, (unsigned long long)q);
+            atomicAdd(g.dense + 3 * k + 2, (unsigned long long)a);
+        }
+    }
+    for (int s = tid; s < kQ1Sparse; s += kQ1Threads)
+        if (sm.stag[s]) q1_global_add(g, sm.stag[s], sm.sacc[s][0], (long long)sm.sacc[s][1],
+                                      (long long)sm.sacc[s][2]);
 }
 
 __global__ void __launch_bounds__(kQ1Threads, 2)
@@ -324,21 +447,96 @@ q1_kernel(const int4 *__restrict__ number, const longlong2 *__restrict__ deliv,
     }
     __syncthreads();
 
-    // merge: dense keys, one warp per key, one global atomic per (key, accumulator) per block
-    const int warp = tid >> 5;
-    for (int k = warp; k < kQ1Dense; k += kQ1Threads / 32) {
-        long long c = 0, q = 0, a = 0;
-        for (int t = lane; t < kQ1Threads; t += 32) { c += sm.cnt[k][t]; q += sm.qty[k][t]; a += sm.amt[k][t]; }
-        c = warp_sum(c); q = warp_sum(q); a = warp_sum(a);
-        if (lane == 0 && c) {
-            atomicAdd(g.dense + 3 * k + 0, (unsigned long long)c);
-            atomicAdd(g.dense + 3 * k + 1, (unsigned long long)q);
-            atomicAdd(g.dense + 3 * k + 2, (unsigned long long)a);
+    q1_block_merge(sm, g, tid);
+}
+
+// Q1, TMA-bulk pipelined variant: one block per SM, warp 8 streams 1024-row chunks of the four
+// columns into a 4-stage ring (96 KB) next to the 88 KB of aggregation tables; warps 0-7
+// aggregate exactly as q1_kernel does (thread-private dense slots, warp-aggregated sparse path).
+constexpr int kQ1Chunk = 1024;
+constexpr int kQ1Stages = 4;
+struct Q1Stages {
+    long long deliv[kQ1Stages][kQ1Chunk];
+    long long amt[kQ1Stages][kQ1Chunk];
+    int number[kQ1Stages][kQ1Chunk];
+    int qty[kQ1Stages][kQ1Chunk];
+    uint64_t full[kQ1Stages], empty[kQ1Stages];
+};
+
+__global__ void __launch_bounds__(kTmaThreads, 1)
+q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deliv,
+              const int *__restrict__ qty, const long long *__restrict__ amt, uint64_t n,
+              long long cutoff, Q1Scratch g) {
+    extern __shared__ __align__(128) unsigned char smem_raw[];
+    Q1Stages &P = *reinterpret_cast<Q1Stages *>(smem_raw);
+    Q1Smem &sm = *reinterpret_cast<Q1Smem *>(smem_raw + sizeof(Q1Stages));
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    if (tid < kQ1Threads) {
+#pragma unroll
+        for (int k = 0; k < kQ1Dense; ++k) { sm.cnt[k][tid] = 0; sm.qty[k][tid] = 0; sm.amt[k][tid] = 0; }
+        for (int s = tid; s < kQ1Sparse; s += kQ1Threads) {
+            sm.stag[s] = 0; sm.sacc[s][0] = 0; sm.sacc[s][1] = 0; sm.sacc[s][2] = 0;
         }
     }
-    for (int s = tid; s < kQ1Sparse; s += kQ1Threads)
-        if (sm.stag[s]) q1_global_add(g, sm.stag[s], sm.sacc[s][0], (long long)sm.sacc[s][1],
-                                      (long long)sm.sacc[s][2]);
+    if (tid == 0) {
+        for (int s = 0; s < kQ1Stages; ++s) {
+            mbar_init(&P.full[s], 1);
+            mbar_init(&P.empty[s], kTmaConsumerWarps);
+        }
+        fence_mbar_init();
+        if (blockIdx.x == 0) *g.ngroups = 0;  // consumed by q1_compact (stream-ordered)
+    }
+    __syncthreads();
+    const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
+    if (warp == kTmaConsumerWarps) {  // producer
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            int it = 0;
+            for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
+                const int s = it % kQ1Stages;
+                const unsigned ph = (unsigned)(it / kQ1Stages) & 1u;
+                if (it >= kQ1Stages) mbar_wait(&P.empty[s], ph ^ 1u);
+                const uint64_t r0 = c * kQ1Chunk;
+                const unsigned rows = (unsigned)(n - r0 < (uint64_t)kQ1Chunk ? n - r0 : (uint64_t)kQ1Chunk);
+                const unsigned b8 = round16(rows * 8), b4 = round16(rows * 4);
+                mbar_arrive_expect_tx(&P.full[s], 2 * b8 + 2 * b4);
+                bulk_g2s(P.deliv[s], deliv + r0, b8, &P.full[s], pol);
+                bulk_g2s(P.amt[s], amt + r0, b8, &P.full[s], pol);
+                bulk_g2s(P.number[s], number + r0, b4, &P.full[s], pol);
+                bulk_g2s(P.qty[s], qty + r0, b4, &P.full[s], pol);
+            }
+        }
+    } else {  // consumers: 256 threads, 4 rows each per chunk (warp-uniform trip count)
+        int it = 0;
+        for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
+            const int s = it % kQ1Stages;
+            mbar_wait(&P.full[s], (unsigned)(it / kQ1Stages) & 1u);
+            const unsigned rows = (unsigned)(n - c * kQ1Chunk < (uint64_t)kQ1Chunk ? n - c * kQ1Chunk
+                                                                                 : (uint64_t)kQ1Chunk);
+#pragma unroll
+            for (int u = 0; u < kQ1Chunk / kQ1Threads; ++u) {
+                const unsigned r = u * kQ1Threads + tid;
+                const bool valid = r < rows;
+                const int key = valid ? P.number[s][r] : 0;
+                const long long d = valid ? P.deliv[s][r] : kNullTs;
+                const int q = valid ? P.qty[s][r] : 0;
+                const long long a = valid ? P.amt[s][r] : 0;
+                // WHERE ol_delivery_d > cutoff (NULL -> UNKNOWN -> excluded), GROUP BY ol_number
+                const bool pass = valid & (d != kNullTs) & (d > cutoff);
+                const bool sparse = pass & ((unsigned)key >= (unsigned)kQ1Dense);
+                if (pass & ((unsigned)key < (unsigned)kQ1Dense)) {
+                    sm.cnt[key][tid] += 1;
+                    sm.qty[key][tid] += q;
+                    sm.amt[key][tid] += a;
+                }
+                if (__any_sync(kFull, sparse)) q1_sparse_warp(sm, g, sparse, key, q, a);
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&P.empty[s]);
+        }
+    }
+    __syncthreads();
+    q1_block_merge(sm, g, tid);
 }
 
 // Collect the dense and global tables into groups[] and clear them for the next query.
@@ -425,6 +623,23 @@ void launch_q6(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uin
         count_launches(1);
 }
 
+void launch_q6_tma(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uint64_t n,
+                   int64_t d_lo, int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s,
+                   int num_sms, cudaStream_t st) {
+    static bool init = false;
+    if (!init) {
+        cudaFuncSetAttribute(q6_tma_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             (int)sizeof(Q6TmaSmem));
+        init = true;
+    }
+    const uint64_t nchunks = (n + kQ6Chunk - 1) / kQ6Chunk;
+    const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
+    q6_tma_kernel<<<grid, kTmaThreads, sizeof(Q6TmaSmem), st>>>(
+        reinterpret_cast<const long long *>(deliv), qty, reinterpret_cast<const long long *>(amt), n,
+        Q6Pred{d_lo, d_hi, q_lo, q_hi}, s.block_part, s.done_counter, s.out);
+    count_launches(1);
+}
+
 void launch_q1_reset(const Q1Scratch &s, cudaStream_t st) {
     cudaMemsetAsync(s.dense, 0, sizeof(unsigned long long) * kQ1Dense * 3, st);
     cudaMemsetAsync(s.gtag, 0, sizeof(unsigned long long) * kQ1GlobalSlots, st);
@@ -450,6 +665,22 @@ void launch_q1(const int32_t *number, const int64_t *deliv, const int32_t *qty,
         reinterpret_cast<const int4 *>(qty), reinterpret_cast<const longlong2 *>(amt), n, cutoff,
         s);
         count_launches(1);
+}
+
+void launch_q1_tma(const int32_t *number, const int64_t *deliv, const int32_t *qty,
+                   const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int num_sms,
+                   cudaStream_t st) {
+    const size_t smem = sizeof(Q1Stages) + sizeof(Q1Smem);
+    static bool init = false;
+    if (!init) {
+        cudaFuncSetAttribute(q1_tma_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        init = true;
+    }
+    const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
+    const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
+    q1_tma_kernel<<<grid, kTmaThreads, smem, st>>>(number, reinterpret_cast<const long long *>(deliv), qty,
+                                                   reinterpret_cast<const long long *>(amt), n, cutoff, s);
+    count_launches(1);
 }
 
 void launch_q1_compact(const Q1Scratch &s, cudaStream_t st) {

@@ -88,3 +88,20 @@ def test_no_oracle_in_product_path():
                 txt = open(os.path.join(dirpath, f)).read()
                 assert "import oracle" not in txt and "from oracle" not in txt, f
                 assert "oracle.h" not in txt and "liboracle" not in txt, f
+
+
+def test_sass_is_sm100a_with_tma_bulk_copies(h):
+    """The library is built for sm_100a only, and the scan kernels stream columns with TMA bulk
+    copies (SASS UBLKCP from cp.async.bulk; B200_PROFILING.md 'What proves a Blackwell-native
+    kernel')."""
+    import shutil
+    import subprocess
+    cuobjdump = shutil.which("cuobjdump") or "/usr/local/cuda/bin/cuobjdump"
+    if not os.path.exists(cuobjdump):
+        pytest.skip("cuobjdump not available")
+    sass = subprocess.run([cuobjdump, "-sass", h.LIB_PATH], capture_output=True, text=True).stdout
+    archs = set(re.findall(r"arch = (sm_\w+)", sass))
+    assert archs == {"sm_100a"}, archs
+    assert "UBLKCP" in sass
+    funcs = re.findall(r"Function : (\S+)", sass)
+    assert any("q6_tma_kernel" in f for f in funcs) and any("q1_tma_kernel" in f for f in funcs)
