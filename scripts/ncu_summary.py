@@ -57,6 +57,8 @@ if traffic:
     json.dump(per, open(tj, "w"), indent=1)
     # per-launch DRAM bytes keyed by the engine's profile marks (what bench.py reports)
     marks = {"q6_kernel": "q6_scan_filter_sum", "q1_kernel": "q1_scan_filter_groupby",
+             "q6_tma_kernel": "q6_scan_filter_sum", "q1_tma_kernel": "q1_scan_filter_groupby",
+             "q18_probe_tma_kernel": "q18_probe_groupjoin",
              "q18_init_kernel": "q18_init", "q18_build_kernel": "q18_build",
              "q18_probe_kernel": "q18_probe_groupjoin", "q18_having_kernel": "q18_having_compact",
              "q18_keys_hist_kernel": "q18_sort_keys_hist", "bucket_scatter_kernel": "q18_bucket_scatter",
