@@ -27,6 +27,7 @@ the same slice of a full generation — the basis of sharding across ranks.
 from __future__ import annotations
 
 import datetime as _dt
+from collections import deque
 from dataclasses import dataclass, field
 
 import numpy as np
@@ -35,7 +36,7 @@ __all__ = [
     "Scale", "TINY", "FULL", "NULL_TS", "LOAD_TS", "TS_1995", "TS_2025",
     "DAY_US", "ts_us", "generate", "generate_item", "neworder_delta",
     "warehouse_ranges", "concat_tables", "TABLE_COLUMNS", "NewOrderState", "neworder_batch",
-    "ROW_DTYPES", "to_records",
+    "ROW_DTYPES", "to_records", "DeliveryState", "delivery_inputs", "delivery_batch",
 ]
 
 
@@ -319,3 +320,65 @@ def to_records(table: str, cols: dict) -> np.ndarray:
     for c in ROW_DTYPES[table].names:
         rec[c] = cols[c]
     return rec
+
+
+# ------------------------------------------------------------------ Delivery --
+@dataclass
+class DeliveryState:
+    """The OLTP side's new_order table: per district (w, d), a FIFO of the undelivered orders in
+    o_id order, each as (o_id, orders row, first order_line row, ol_cnt) — row positions in the
+    host row store, which is what an in-place update names (NEXT-1).
+
+    ``add(orders, o_row0, ol_row0)`` registers a block of orders stored at orders rows
+    ``o_row0 + i`` whose lines are stored contiguously, in the same order, from order_line row
+    ``ol_row0`` on (true for ``generate`` tables and for ``neworder_batch`` deltas)."""
+    districts: int = FULL.districts
+    queues: dict = field(default_factory=dict)
+
+    def add(self, orders: dict, o_row0: int = 0, ol_row0: int = 0):
+        cnt = orders["o_ol_cnt"].astype(np.int64)
+        ol_first = ol_row0 + np.concatenate([[0], np.cumsum(cnt)[:-1]]) if len(cnt) else cnt
+        pending = np.flatnonzero(orders["o_carrier_id"] == -1)
+        w, d, o = orders["o_w_id"], orders["o_d_id"], orders["o_id"]
+        for i in pending.tolist():
+            self.queues.setdefault((int(w[i]), int(d[i])), deque()).append(
+                (int(o[i]), o_row0 + i, int(ol_first[i]), int(cnt[i])))
+
+    def undelivered(self) -> int:
+        return sum(len(q) for q in self.queues.values())
+
+
+def delivery_inputs(n_txn: int, *, seed: int, batch: int, w_lo: int, w_hi: int):
+    """The random inputs of ``n_txn`` TPC-C Delivery transactions (TPC-C 2.7.1 [EXT]): home
+    warehouse uniform in [w_lo, w_hi), o_carrier_id uniform in [1, 10]."""
+    rng = np.random.Generator(np.random.Philox(key=np.array([seed, 1 << 42 | batch], dtype=np.uint64)))
+    w = rng.integers(w_lo, w_hi, size=n_txn).astype(np.int32)
+    carrier = rng.integers(1, 11, size=n_txn).astype(np.int32)
+    return w, carrier
+
+
+def delivery_batch(state: DeliveryState, w, carrier, clock0: int, step_us: int = 1_000):
+    """Row updates of Delivery transactions (TPC-C 2.7.4 [EXT], as SURVEY.md §8(f) NEXT-1 uses it):
+    transaction k runs at time ``clock0 + (k+1)*step_us``; for each district d of warehouse
+    ``w[k]`` it takes the oldest undelivered order (if any), sets its o_carrier_id to
+    ``carrier[k]`` and the ol_delivery_d of each of its lines to the transaction time.
+    (The customer balance / delivery count updates touch no column of the hot path.)
+
+    Returns ``{"orders": {"o_carrier_id": (rows, values)},
+    "order_line": {"ol_delivery_d": (rows, values)}}`` with rows uint32 (distinct: an order is
+    delivered once) and values in the column dtype."""
+    o_rows, o_vals, l_rows, l_vals = [], [], [], []
+    for k in range(len(w)):
+        ts = clock0 + (k + 1) * step_us
+        for d in range(1, state.districts + 1):
+            q = state.queues.get((int(w[k]), d))
+            if not q:
+                continue
+            _, o_row, ol_first, cnt = q.popleft()
+            o_rows.append(o_row)
+            o_vals.append(int(carrier[k]))
+            l_rows.extend(range(ol_first, ol_first + cnt))
+            l_vals.extend([ts] * cnt)
+    return {"orders": {"o_carrier_id": (np.asarray(o_rows, np.uint32), np.asarray(o_vals, np.int32))},
+            "order_line": {"ol_delivery_d": (np.asarray(l_rows, np.uint32),
+                                             np.asarray(l_vals, np.int64))}}

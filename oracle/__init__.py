@@ -157,3 +157,19 @@ def q18(tables, having):
         if n <= cap:
             return {k: v[:n] for k, v in out.items()}
         cap = n
+
+
+def apply_updates(tables, updates):
+    """The snapshot after in-place updates: for every
+    ``updates[table][column] = (rows, values)``, row ``rows[i]`` of that column holds
+    ``values[i]``; every other value is unchanged. This is the plain definition of the paper's
+    copy-on-write update as seen by a later snapshot ("updates ... shadow-copy the pages they
+    touch"); row ids are distinct. Returns new tables; the input tables (the
+    previous snapshot) are not modified."""
+    out = {t: dict(cols) for t, cols in tables.items()}
+    for t, per_col in updates.items():
+        for c, (rows, values) in per_col.items():
+            col = np.array(out[t][c], copy=True)
+            col[np.asarray(rows, dtype=np.int64)] = values
+            out[t][c] = col
+    return out

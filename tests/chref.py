@@ -43,16 +43,18 @@ def sqlite_load(tables):
     db.execute("CREATE TABLE order_line (ol_w_id INT, ol_d_id INT, ol_o_id INT, ol_number INT,"
                " ol_delivery_d INT, ol_quantity INT, ol_amount INT)")
     db.execute("CREATE TABLE orders (o_w_id INT, o_d_id INT, o_id INT, o_c_id INT, o_ol_cnt INT,"
-               " o_entry_d INT)")
+               " o_entry_d INT, o_carrier_id INT)")
     db.execute("CREATE TABLE customer (c_w_id INT, c_d_id INT, c_id INT, c_last INT)")
     deliv = [None if int(v) == NULL_SENTINEL else int(v) for v in ol["ol_delivery_d"]]
     db.executemany("INSERT INTO order_line VALUES (?,?,?,?,?,?,?)",
                    zip(ol["ol_w_id"].tolist(), ol["ol_d_id"].tolist(), ol["ol_o_id"].tolist(),
                        ol["ol_number"].tolist(), deliv, ol["ol_quantity"].tolist(),
                        ol["ol_amount"].tolist()))
-    db.executemany("INSERT INTO orders VALUES (?,?,?,?,?,?)",
+    carrier = [None if int(v) == -1 else int(v) for v in o["o_carrier_id"]]
+    db.executemany("INSERT INTO orders VALUES (?,?,?,?,?,?,?)",
                    zip(o["o_w_id"].tolist(), o["o_d_id"].tolist(), o["o_id"].tolist(),
-                       o["o_c_id"].tolist(), o["o_ol_cnt"].tolist(), o["o_entry_d"].tolist()))
+                       o["o_c_id"].tolist(), o["o_ol_cnt"].tolist(), o["o_entry_d"].tolist(),
+                       carrier))
     db.executemany("INSERT INTO customer VALUES (?,?,?,?)",
                    zip(c["c_w_id"].tolist(), c["c_d_id"].tolist(), c["c_id"].tolist(),
                        c["c_last"].tolist()))
@@ -86,6 +88,27 @@ def sqlite_q18(db, having):
         "GROUP BY o_id, o_w_id, o_d_id, c_id, c_last, o_entry_d, o_ol_cnt "
         "HAVING SUM(ol_amount) > ? ORDER BY amount_sum DESC, o_entry_d",
         (having,)).fetchall()
+
+
+def sqlite_delivery(db, w, carrier, ts, districts):
+    """One TPC-C Delivery transaction (TPC-C 2.7.4.2 [EXT]) as SQL: for each district, the
+    oldest undelivered order (new_order = orders with a NULL carrier) gets the carrier and its
+    lines get delivery date ts."""
+    for d in range(1, districts + 1):
+        (o,) = db.execute("SELECT MIN(o_id) FROM orders WHERE o_w_id = ? AND o_d_id = ? "
+                          "AND o_carrier_id IS NULL", (w, d)).fetchone()
+        if o is None:
+            continue
+        db.execute("UPDATE orders SET o_carrier_id = ? WHERE o_w_id = ? AND o_d_id = ? AND o_id = ?",
+                   (carrier, w, d, o))
+        db.execute("UPDATE order_line SET ol_delivery_d = ? "
+                   "WHERE ol_w_id = ? AND ol_d_id = ? AND ol_o_id = ?", (ts, w, d, o))
+
+
+def sqlite_column(db, table, column, null):
+    """A column in insertion (rowid) order, SQL NULL mapped back to the sentinel ``null``."""
+    return [null if v is None else v
+            for (v,) in db.execute(f"SELECT {column} FROM {table} ORDER BY rowid")]
 
 
 # -------------------------------------------------------------- brute force --
