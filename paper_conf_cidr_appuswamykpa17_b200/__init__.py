@@ -6,6 +6,7 @@ the query kernels, the NCCL merge and the finalisation all run in the CUDA libra
 no CPU fallback — importing this package fails loudly when the library is missing.
 
 Names mirror the ABI: ``h2tap_open``, ``h2tap_load_snapshot``, ``h2tap_sync``,
+``h2tap_refresh``, ``h2tap_refresh_rows``, ``h2tap_get_store_stats``,
 ``h2tap_run_query``, ``h2tap_free``, ``h2tap_close``, ``h2tap_last_error``,
 ``h2tap_nccl_unique_id``, ``h2tap_compute_stream``, ``h2tap_c_last_name``.
 """
@@ -77,6 +78,19 @@ class h2tap_row_table(C.Structure):
                 ("first_row", C.c_uint64), ("flags", C.c_uint32)]
 
 
+class h2tap_update(C.Structure):
+    _fields_ = [("table_id", C.c_uint32), ("column_id", C.c_uint32), ("type", C.c_uint32),
+                ("n", C.c_uint64), ("row_ids", C.c_void_p), ("values", C.c_void_p)]
+
+
+class h2tap_store_stats(C.Structure):
+    _fields_ = [("published_epoch", C.c_uint64), ("refreshes", C.c_uint64),
+                ("rows_appended", C.c_uint64), ("rows_updated", C.c_uint64),
+                ("cow_pages_copied", C.c_uint64), ("cow_full_copies", C.c_uint64),
+                ("device_bytes", C.c_uint64), ("last_load_ms", C.c_double),
+                ("last_update_ms", C.c_double)]
+
+
 class h2tap_config(C.Structure):
     _fields_ = [("device", C.c_int), ("rank", C.c_int), ("world", C.c_int),
                 ("nccl_unique_id", C.c_void_p)]
@@ -105,6 +119,11 @@ _lib.h2tap_sync.argtypes = [_P, C.POINTER(C.c_uint64)]
 _lib.h2tap_reserve.argtypes = [_P, C.c_uint32, C.c_uint64]
 _lib.h2tap_load_snapshot_rows.argtypes = [_P, C.POINTER(h2tap_row_table), C.c_uint32, C.c_uint64,
                                           C.c_uint32]
+_lib.h2tap_refresh.argtypes = [_P, C.POINTER(h2tap_table), C.c_uint32, C.POINTER(h2tap_update),
+                               C.c_uint32, C.c_uint64, C.c_uint32]
+_lib.h2tap_refresh_rows.argtypes = [_P, C.POINTER(h2tap_row_table), C.c_uint32,
+                                    C.POINTER(h2tap_update), C.c_uint32, C.c_uint64, C.c_uint32]
+_lib.h2tap_get_store_stats.argtypes = [_P, C.POINTER(h2tap_store_stats)]
 _lib.h2tap_run_query_ex.argtypes = [_P, C.c_uint32, C.POINTER(C.c_int64), C.c_uint32, C.c_uint32,
                                     C.POINTER(C.POINTER(h2tap_result))]
 _lib.h2tap_run_query.argtypes = [_P, C.c_uint32, C.POINTER(C.c_int64), C.c_uint32,
@@ -120,14 +139,15 @@ _lib.h2tap_nccl_unique_id.argtypes = [_P]
 _lib.h2tap_compute_stream.argtypes = [_P, C.POINTER(_P)]
 _lib.h2tap_c_last_name.argtypes = [C.c_int32, C.c_char_p, C.c_size_t]
 for _f in ("h2tap_open", "h2tap_load_snapshot_ex", "h2tap_load_snapshot", "h2tap_load_snapshot_rows",
-           "h2tap_reserve",
+           "h2tap_reserve", "h2tap_refresh", "h2tap_refresh_rows", "h2tap_get_store_stats",
            "h2tap_sync",
            "h2tap_run_query_ex", "h2tap_run_query", "h2tap_run_queries", "h2tap_nccl_unique_id",
            "h2tap_compute_stream"):
     getattr(_lib, _f).restype = C.c_int
 
 ABI_SYMBOLS = ["h2tap_open", "h2tap_load_snapshot", "h2tap_load_snapshot_ex",
-               "h2tap_load_snapshot_rows", "h2tap_reserve", "h2tap_sync",
+               "h2tap_load_snapshot_rows", "h2tap_reserve", "h2tap_refresh", "h2tap_refresh_rows",
+               "h2tap_get_store_stats", "h2tap_sync",
                "h2tap_run_query", "h2tap_run_query_ex", "h2tap_run_queries", "h2tap_free", "h2tap_close",
                "h2tap_last_error", "h2tap_nccl_unique_id", "h2tap_compute_stream",
                "h2tap_c_last_name"]
@@ -196,15 +216,7 @@ def _host_ptr(a, want_dtype, name):
     return arr.ctypes.data, arr, arr.size
 
 
-def h2tap_load_snapshot(engine: Engine, tables: dict, epoch: int, *, flags: int = 0,
-                        full_reload=True, first_row: dict | None = None) -> None:
-    """Refresh the device snapshot to ``epoch``.
-
-    ``tables``: {table_name: {column_name: array}} with the generator's names. Each array holds
-    rows [first_row, row_count) of its column. ``full_reload`` (bool, or a set of table names)
-    replaces those tables; other tables are appended to (``first_row[table]`` = rows already
-    loaded). ``flags``: H2TAP_LOAD_ASYNC to return before the epoch is published.
-    """
+def _column_tables(tables, full_reload, first_row):
     first_row = first_row or {}
     keep, tabs, colarrs = [], [], []
     for tname, cols in tables.items():
@@ -226,17 +238,58 @@ def h2tap_load_snapshot(engine: Engine, tables: dict, epoch: int, *, flags: int 
         colarrs.append(carr)
         tabs.append(h2tap_table(tid, len(cols), carr, fr + (nrows or 0), fr,
                                 H2TAP_FULL_RELOAD if full else 0))
-    tarr = (h2tap_table * len(tabs))(*tabs)
-    _check(_lib.h2tap_load_snapshot_ex(engine.handle, tarr, len(tabs), epoch, flags))
-    del keep, colarrs
+    return (h2tap_table * len(tabs))(*tabs), len(tabs), keep + colarrs
 
 
-def h2tap_load_snapshot_rows(engine: Engine, tables: dict, epoch: int, *, flags: int = 0,
-                             full_reload=True, first_row: dict | None = None,
-                             columns: dict | None = None) -> None:
-    """Refresh from a host ROW store: ``tables`` = {table_name: numpy structured array of NSM
-    records}. ``columns`` optionally restricts the extracted fields per table (default: every
-    schema field present in the record dtype). Other arguments as h2tap_load_snapshot."""
+def _updates(updates):
+    """{table: {column: (row_ids, values)}} -> h2tap_update array (+ objects to keep alive)."""
+    ups, keep = [], []
+    for tname, per_col in (updates or {}).items():
+        tid, schema = SCHEMA[tname]
+        ids = {n: (i, t) for i, (n, t) in enumerate(schema)}
+        for cname, (rows, vals) in per_col.items():
+            cid, ty = ids[cname]
+            rp, robj, nr = _host_ptr(rows, np.uint32, f"{tname}.{cname} row ids")
+            vp, vobj, nv = _host_ptr(vals, _DT[ty], f"{tname}.{cname} values")
+            if nr != nv:
+                raise ValueError(f"{tname}.{cname}: {nr} row ids but {nv} values")
+            keep += [robj, vobj]
+            ups.append(h2tap_update(tid, cid, ty, nr, rp if nr else None, vp if nv else None))
+    return (h2tap_update * max(len(ups), 1))(*ups), len(ups), keep
+
+
+def h2tap_load_snapshot(engine: Engine, tables: dict, epoch: int, *, flags: int = 0,
+                        full_reload=True, first_row: dict | None = None) -> None:
+    """Refresh the device snapshot to ``epoch``.
+
+    ``tables``: {table_name: {column_name: array}} with the generator's names. Each array holds
+    rows [first_row, row_count) of its column. ``full_reload`` (bool, or a set of table names)
+    replaces those tables; other tables are appended to (``first_row[table]`` = rows already
+    loaded). ``flags``: H2TAP_LOAD_ASYNC to return before the epoch is published.
+    """
+    tarr, nt, keep = _column_tables(tables, full_reload, first_row)
+    _check(_lib.h2tap_load_snapshot_ex(engine.handle, tarr, nt, epoch, flags))
+    del keep
+
+
+def h2tap_refresh(engine: Engine, tables: dict | None, updates: dict | None, epoch: int, *,
+                  flags: int = 0, full_reload=False, first_row: dict | None = None) -> None:
+    """One new epoch = appends / reloads of ``tables`` (as h2tap_load_snapshot; default append)
+    then in-place ``updates`` = {table: {column: (row_ids uint32, values)}} (copy-on-write)."""
+    tarr, nt, keep = _column_tables(tables or {}, full_reload, first_row)
+    uarr, nu, ukeep = _updates(updates)
+    _check(_lib.h2tap_refresh(engine.handle, tarr, nt, uarr, nu, epoch, flags))
+    del keep, ukeep
+
+
+def h2tap_get_store_stats(engine: Engine) -> dict:
+    """Snapshot-store counters and the last refresh's copy-stream times (h2tap_store_stats)."""
+    st = h2tap_store_stats()
+    _check(_lib.h2tap_get_store_stats(engine.handle, C.byref(st)))
+    return {name: getattr(st, name) for name, _ in h2tap_store_stats._fields_}
+
+
+def _row_tables(tables, full_reload, first_row, columns):
     first_row = first_row or {}
     keep, tabs = [], []
     for tname, rec in tables.items():
@@ -258,9 +311,28 @@ def h2tap_load_snapshot_rows(engine: Engine, tables: dict, epoch: int, *, flags:
         tabs.append(h2tap_row_table(tid, len(fields), farr, rec.ctypes.data if len(rec) else None,
                                     rec.dtype.itemsize, fr + len(rec), fr,
                                     H2TAP_FULL_RELOAD if full else 0))
-    tarr = (h2tap_row_table * len(tabs))(*tabs)
-    _check(_lib.h2tap_load_snapshot_rows(engine.handle, tarr, len(tabs), epoch, flags))
+    return (h2tap_row_table * len(tabs))(*tabs), len(tabs), keep
+
+
+def h2tap_load_snapshot_rows(engine: Engine, tables: dict, epoch: int, *, flags: int = 0,
+                             full_reload=True, first_row: dict | None = None,
+                             columns: dict | None = None) -> None:
+    """Refresh from a host ROW store: ``tables`` = {table_name: numpy structured array of NSM
+    records}. ``columns`` optionally restricts the extracted fields per table (default: every
+    schema field present in the record dtype). Other arguments as h2tap_load_snapshot."""
+    tarr, nt, keep = _row_tables(tables, full_reload, first_row, columns)
+    _check(_lib.h2tap_load_snapshot_rows(engine.handle, tarr, nt, epoch, flags))
     del keep
+
+
+def h2tap_refresh_rows(engine: Engine, tables: dict | None, updates: dict | None, epoch: int, *,
+                       flags: int = 0, full_reload=False, first_row: dict | None = None,
+                       columns: dict | None = None) -> None:
+    """h2tap_load_snapshot_rows (default append) plus in-place ``updates`` in the same epoch."""
+    tarr, nt, keep = _row_tables(tables or {}, full_reload, first_row, columns)
+    uarr, nu, ukeep = _updates(updates)
+    _check(_lib.h2tap_refresh_rows(engine.handle, tarr, nt, uarr, nu, epoch, flags))
+    del keep, ukeep
 
 
 def h2tap_reserve(engine: Engine, table: str, rows: int) -> None:

@@ -208,8 +208,13 @@ struct View {  // immutable snapshot at one epoch (the paper's shallow-copied to
 using ViewP = std::shared_ptr<const View>;
 
 struct ColState {
-    DevBufP cur, spare;
+    // cur: the latest accepted version. alt: the shadow (an earlier version, or a spare for full
+    // reloads); when alt_valid, alt equals cur on rows [0, alt_synced) except on the pages whose
+    // bit is set in `bits` (copy-on-write of in-place updates, store_kernels.cu)
+    DevBufP cur, alt, bits;
     uint64_t cap_rows = 0;
+    bool alt_valid = false;
+    uint64_t alt_synced = 0;
 };
 struct TableState {
     bool present = false;
@@ -222,10 +227,14 @@ struct Pending {
     uint64_t epoch;
     std::shared_ptr<View> view;   // becomes visible (const) at publish
     cudaEvent_t done;
-    bool loaded[kTables], full[kTables];
-    int *stats_host;              // pinned [kTables][kStatCols][2] delta min/max
+    cudaEvent_t t0, t1, t2;       // timing: begin, loads done, updates done (copy stream)
+    bool loaded[kTables], full[kTables], updated[kTables];
+    int *stats_host;              // pinned [kTables][kStatCols][2] delta min/max, then the u64
+                                  // count of pages copied into shadows (kStatBytes offset)
     std::pair<void *, size_t> stats_block;
+    uint64_t rows_appended, rows_updated, full_copies;
 };
+constexpr size_t kStatBytes = sizeof(int) * kTables * kStatCols * 2;  // multiple of 8
 
 struct Staging {  // pinned ring for pageable host buffers
     static constexpr size_t kChunk = 32u << 20;
@@ -298,6 +307,7 @@ struct h2tap_engine {
     std::deque<Pending> pending;
     Staging staging;
 
+    h2tap_store_stats sstats{};  // under pend_mu
     Arena arena;       // query scratch (compute stream)
     Arena load_arena;  // refresh scratch (copy stream)
     Prof prof;
@@ -325,21 +335,37 @@ void publish_ready(h2tap_engine *e, bool wait) {
                 for (int c = 0; c < kStatCols; ++c) {
                     int mn = INT32_MAX, mx = INT32_MIN;
                     if (carry) { mn = prev->smin[t][c]; mx = prev->smax[t][c]; }
-                    if (p.loaded[t]) {
+                    if (p.loaded[t] || p.updated[t]) {
                         mn = std::min(mn, p.stats_host[(t * kStatCols + c) * 2]);
                         mx = std::max(mx, p.stats_host[(t * kStatCols + c) * 2 + 1]);
                     }
                     v.smin[t][c] = mn;
                     v.smax[t][c] = mx;
                 }
-                v.has_stats[t] = p.loaded[t] || carry;
+                v.has_stats[t] = p.loaded[t] || p.updated[t] || carry;
             }
+        }
+        {
+            h2tap_store_stats &S = e->sstats;
+            S.published_epoch = p.epoch;
+            S.refreshes += 1;
+            S.rows_appended += p.rows_appended;
+            S.rows_updated += p.rows_updated;
+            S.cow_full_copies += p.full_copies;
+            uint64_t pages;
+            std::memcpy(&pages, reinterpret_cast<char *>(p.stats_host) + kStatBytes, 8);
+            S.cow_pages_copied += pages;
+            float a = 0, b = 0;
+            CK(cudaEventElapsedTime(&a, p.t0, p.t1));
+            CK(cudaEventElapsedTime(&b, p.t1, p.t2));
+            S.last_load_ms = a;
+            S.last_update_ms = b;
         }
         {
             std::lock_guard<std::mutex> gv(e->view_mu);
             e->published = p.view;
         }
-        cudaEventDestroy(p.done);
+        for (cudaEvent_t ev : {p.done, p.t0, p.t1, p.t2}) cudaEventDestroy(ev);
         e->host_pool->put(p.stats_block.first, p.stats_block.second);
         e->pending.pop_front();
     }
@@ -383,7 +409,8 @@ bool h2d(h2tap_engine *e, void *dst, const void *src, size_t bytes) {
 }
 
 h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntables,
-                       uint64_t epoch, uint32_t flags) {
+                       const h2tap_update *updates, uint32_t nupdates, uint64_t epoch,
+                       uint32_t flags) {
     std::lock_guard<std::mutex> g(e->load_mu);
     CK(cudaSetDevice(e->device));
     publish_ready(e, false);
@@ -391,6 +418,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         return fail(H2TAP_ESTALE, "epoch %llu is not greater than the last accepted epoch %llu",
                     (unsigned long long)epoch, (unsigned long long)e->last_epoch.load());
     if (ntables && !tables) return fail(H2TAP_EINVAL, "tables is NULL");
+    if (nupdates && !updates) return fail(H2TAP_EINVAL, "updates is NULL");
     // ---- validate everything before touching state
     bool seen[kTables] = {};
     for (uint32_t i = 0; i < ntables; ++i) {
@@ -426,6 +454,41 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
                             t.table_id, (unsigned long long)t.first_row, (unsigned long long)ts.loaded);
         }
     }
+    {  // updates: target columns loaded at the new epoch, row ids inside its row count
+        uint32_t listed[kTables] = {};
+        for (uint32_t i = 0; i < nupdates; ++i) {
+            const h2tap_update &u = updates[i];
+            if (u.table_id < 1 || u.table_id > 4) return fail(H2TAP_EINVAL, "update %u: unknown table id %u", i, u.table_id);
+            if (u.column_id >= (uint32_t)kNcols[u.table_id])
+                return fail(H2TAP_EINVAL, "update %u: unknown column id %u", i, u.column_id);
+            if (u.type != kTypes[u.table_id][u.column_id])
+                return fail(H2TAP_EINVAL, "update %u: type %u, schema type %u", i, u.type,
+                            kTypes[u.table_id][u.column_id]);
+            if (listed[u.table_id] & (1u << u.column_id))
+                return fail(H2TAP_EINVAL, "update %u: table %u column %u listed twice", i, u.table_id, u.column_id);
+            listed[u.table_id] |= 1u << u.column_id;
+            if (u.n && (!u.row_ids || !u.values)) return fail(H2TAP_EINVAL, "update %u: NULL row_ids/values", i);
+            uint32_t mask = 0;
+            uint64_t rows = 0;
+            if (seen[u.table_id]) {
+                for (uint32_t k = 0; k < ntables; ++k)
+                    if (tables[k].table_id == u.table_id) {
+                        for (uint32_t c = 0; c < tables[k].ncols; ++c) mask |= 1u << tables[k].cols[c].column_id;
+                        rows = tables[k].row_count;
+                    }
+            } else if (e->tables[u.table_id].present) {
+                mask = e->tables[u.table_id].colmask;
+                rows = e->accepted ? e->accepted->n[u.table_id] : 0;
+            }
+            if (!(mask & (1u << u.column_id)))
+                return fail(H2TAP_EPLAN, "update %u: table %u column %u was never loaded", i, u.table_id, u.column_id);
+            uint32_t mx = 0;
+            for (uint64_t k = 0; k < u.n; ++k) mx = std::max(mx, u.row_ids[k]);
+            if (u.n && mx >= rows)
+                return fail(H2TAP_EINVAL, "update %u: row id %u outside the table's %llu rows", i, mx,
+                            (unsigned long long)rows);
+        }
+    }
     // ---- copy and build the new view
     auto v = std::make_shared<View>();
     if (e->accepted) *v = *e->accepted;
@@ -433,10 +496,14 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
     bool must_wait = false;
     Pending pend{};
     pend.epoch = epoch;
-    pend.stats_block = e->host_pool->get(sizeof(int) * kTables * kStatCols * 2);
+    pend.stats_block = e->host_pool->get(kStatBytes + 8);
     pend.stats_host = static_cast<int *>(pend.stats_block.first);
-    int *stats_dev = static_cast<int *>(e->load_arena.get("load.stats", sizeof(int) * kTables * kStatCols * 2));
+    int *stats_dev = static_cast<int *>(e->load_arena.get("load.stats", kStatBytes + 8));
+    auto *pages_dev = reinterpret_cast<unsigned long long *>(reinterpret_cast<char *>(stats_dev) + kStatBytes);
+    for (cudaEvent_t *ev : {&pend.t0, &pend.t1, &pend.t2}) CK(cudaEventCreate(ev));
+    CK(cudaEventRecord(pend.t0, e->copy));
     launch_stats_init(stats_dev, kTables * kStatCols, e->copy);
+    CK(cudaMemsetAsync(pages_dev, 0, 8, e->copy));
     for (uint32_t i = 0; i < ntables; ++i) {
         const h2tap_table &t = tables[i];
         TableState &ts = e->tables[t.table_id];
@@ -461,9 +528,10 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
                 // never overwrite a buffer a live view may read: reuse the spare only when no
                 // view references it any more, else allocate
                 DevBufP target;
-                if (cs.spare && cs.spare.use_count() == 1 && cs.spare->bytes >= need * es) target = cs.spare;
+                if (cs.alt && cs.alt.use_count() == 1 && cs.alt->bytes >= need * es) target = cs.alt;
                 else target = dev_alloc(need * es + need * es / 8, e->device);
-                cs.spare = cs.cur;
+                cs.alt = cs.cur;
+                cs.alt_valid = false;
                 cs.cur = target;
                 cs.cap_rows = target->bytes / es;
             } else if (!cs.cur || need > cs.cap_rows) {
@@ -473,7 +541,8 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
                 DevBufP nb = dev_alloc(cap * es, e->device);
                 if (cs.cur && t.first_row)
                     CK(cudaMemcpyAsync(nb->ptr, cs.cur->ptr, t.first_row * es, cudaMemcpyDeviceToDevice, e->copy));
-                cs.spare.reset();
+                cs.alt.reset();
+                cs.alt_valid = false;
                 cs.cur = nb;
                 cs.cap_rows = cap;
             }
@@ -488,6 +557,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
             for (uint32_t c = 0; c < t.ncols; ++c) mask |= 1u << t.cols[c].column_id;
             ts.colmask = mask;
         }
+        pend.rows_appended += t.row_count - t.first_row;
         ts.loaded = t.row_count;
         v->n[t.table_id] = t.row_count;
         pend.loaded[t.table_id] = true;
@@ -500,9 +570,50 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
                                       t.row_count - t.first_row,
                                       stats_dev + (t.table_id * kStatCols + c) * 2, e->num_sms, e->copy);
     }
+    CK(cudaEventRecord(pend.t1, e->copy));
+    // ---- in-place updates: rebuild each updated column in its shadow buffer (copy-on-write)
+    for (uint32_t i = 0; i < nupdates; ++i) {
+        const h2tap_update &u = updates[i];
+        ColState &cs = e->tables[u.table_id].col[u.column_id];
+        const size_t es = type_size(u.type);
+        const uint64_t n_rows = v->n[u.table_id];
+        const uint64_t words = (cs.cap_rows + kCowPageRows * 32 - 1) / (kCowPageRows * 32);
+        if (!cs.bits || cs.bits->bytes < words * 4) {
+            cs.bits = dev_alloc(words * 4, e->device);
+            cs.alt_valid = false;  // no record of where alt differs
+        }
+        uint32_t *bits = static_cast<uint32_t *>(cs.bits->ptr);
+        const bool reuse = cs.alt && cs.alt.use_count() == 1 && cs.alt->bytes >= cs.cap_rows * es;
+        if (reuse && cs.alt_valid) {
+            launch_cow_catchup(cs.alt->ptr, cs.cur->ptr, (uint32_t)es, bits, cs.alt_synced, n_rows,
+                               pages_dev, e->num_sms, e->copy);
+        } else {
+            if (!reuse) cs.alt = dev_alloc(cs.cap_rows * es, e->device);
+            if (n_rows) CK(cudaMemcpyAsync(cs.alt->ptr, cs.cur->ptr, n_rows * es, cudaMemcpyDeviceToDevice, e->copy));
+            pend.full_copies += 1;
+        }
+        CK(cudaMemsetAsync(bits, 0, words * 4, e->copy));
+        if (u.n) {
+            auto *rows_d = static_cast<uint32_t *>(e->load_arena.get("upd.rows", u.n * 4));
+            void *vals_d = e->load_arena.get("upd.vals", u.n * es);
+            must_wait |= h2d(e, rows_d, u.row_ids, u.n * 4);
+            must_wait |= h2d(e, vals_d, u.values, u.n * es);
+            launch_apply_updates(cs.alt->ptr, (uint32_t)es, bits, rows_d, vals_d, u.n, e->num_sms, e->copy);
+            if (u.table_id != H2TAP_T_ITEM && u.column_id < (uint32_t)kStatCols)  // zone map: widen
+                launch_minmax_i32(static_cast<const int32_t *>(vals_d), u.n,
+                                  stats_dev + (u.table_id * kStatCols + u.column_id) * 2, e->num_sms, e->copy);
+        }
+        std::swap(cs.cur, cs.alt);
+        cs.alt_valid = true;
+        cs.alt_synced = n_rows;
+        v->col[u.table_id][u.column_id] = cs.cur->ptr;
+        v->keep[u.table_id][u.column_id] = cs.cur;
+        pend.updated[u.table_id] = true;
+        pend.rows_updated += u.n;
+    }
+    CK(cudaEventRecord(pend.t2, e->copy));
     CK(cudaGetLastError());
-    CK(cudaMemcpyAsync(pend.stats_host, stats_dev, sizeof(int) * kTables * kStatCols * 2,
-                       cudaMemcpyDeviceToHost, e->copy));
+    CK(cudaMemcpyAsync(pend.stats_host, stats_dev, kStatBytes + 8, cudaMemcpyDeviceToHost, e->copy));
     CK(cudaEventCreateWithFlags(&pend.done, cudaEventDisableTiming));
     CK(cudaEventRecord(pend.done, e->copy));
     pend.view = v;
@@ -1176,7 +1287,7 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
 h2tap_status h2tap_load_snapshot_ex(h2tap_engine *e, const h2tap_table *tables, uint32_t ntables,
                                     uint64_t epoch, uint32_t flags) {
     if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
-    return guarded([&] { return load_impl(e, tables, ntables, epoch, flags); });
+    return guarded([&] { return load_impl(e, tables, ntables, nullptr, 0, epoch, flags); });
 }
 
 h2tap_status h2tap_reserve(h2tap_engine *e, uint32_t table_id, uint64_t rows) {
@@ -1194,7 +1305,8 @@ h2tap_status h2tap_reserve(h2tap_engine *e, uint32_t table_id, uint64_t rows) {
             DevBufP nb = dev_alloc(need * es, e->device);
             if (ts.loaded)
                 CK(cudaMemcpyAsync(nb->ptr, cs.cur->ptr, ts.loaded * es, cudaMemcpyDeviceToDevice, e->copy));
-            cs.spare.reset();
+            cs.alt.reset();
+            cs.alt_valid = false;
             cs.cur = nb;  // published views keep the old buffer alive until they retire
             cs.cap_rows = need;
         }
@@ -1203,8 +1315,36 @@ h2tap_status h2tap_reserve(h2tap_engine *e, uint32_t table_id, uint64_t rows) {
     });
 }
 
-h2tap_status h2tap_load_snapshot_rows(h2tap_engine *e, const h2tap_row_table *tables,
-                                      uint32_t ntables, uint64_t epoch, uint32_t flags) {
+h2tap_status h2tap_refresh(h2tap_engine *e, const h2tap_table *tables, uint32_t ntables,
+                           const h2tap_update *updates, uint32_t nupdates, uint64_t epoch,
+                           uint32_t flags) {
+    if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
+    return guarded([&] { return load_impl(e, tables, ntables, updates, nupdates, epoch, flags); });
+}
+
+h2tap_status h2tap_get_store_stats(h2tap_engine *e, h2tap_store_stats *out) {
+    if (!e || !out) return fail(H2TAP_EINVAL, "NULL argument");
+    return guarded([&]() -> h2tap_status {
+        std::lock_guard<std::mutex> g(e->load_mu);
+        CK(cudaSetDevice(e->device));
+        publish_ready(e, false);
+        {
+            std::lock_guard<std::mutex> gp(e->pend_mu);
+            *out = e->sstats;
+        }
+        uint64_t bytes = 0;
+        for (auto &t : e->tables)
+            for (auto &c : t.col)
+                for (const DevBufP *b : {&c.cur, &c.alt, &c.bits})
+                    if (*b) bytes += (*b)->bytes;
+        out->device_bytes = bytes;
+        return H2TAP_OK;
+    });
+}
+
+h2tap_status h2tap_refresh_rows(h2tap_engine *e, const h2tap_row_table *tables, uint32_t ntables,
+                                const h2tap_update *updates, uint32_t nupdates, uint64_t epoch,
+                                uint32_t flags) {
     if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
     if (ntables && !tables) return fail(H2TAP_EINVAL, "tables is NULL");
     return guarded([&]() -> h2tap_status {
@@ -1254,8 +1394,13 @@ h2tap_status h2tap_load_snapshot_rows(h2tap_engine *e, const h2tap_row_table *ta
         work(0);
         for (auto &th : pool) th.join();
         // pinned sources: load_impl DMAs them directly and waits before returning
-        return load_impl(e, tabs.data(), ntables, epoch, flags);
+        return load_impl(e, tabs.data(), ntables, updates, nupdates, epoch, flags);
     });
+}
+
+h2tap_status h2tap_load_snapshot_rows(h2tap_engine *e, const h2tap_row_table *tables,
+                                      uint32_t ntables, uint64_t epoch, uint32_t flags) {
+    return h2tap_refresh_rows(e, tables, ntables, nullptr, 0, epoch, flags);
 }
 
 h2tap_status h2tap_load_snapshot(h2tap_engine *e, const h2tap_table *tables, uint32_t ntables,
@@ -1304,7 +1449,7 @@ void h2tap_close(h2tap_engine *e) {
     cudaStreamSynchronize(e->copy);
     if (e->comm) ncclCommDestroy(e->comm);
     for (auto &p : e->pending) {
-        cudaEventDestroy(p.done);
+        for (cudaEvent_t ev : {p.done, p.t0, p.t1, p.t2}) cudaEventDestroy(ev);
         e->host_pool->put(p.stats_block.first, p.stats_block.second);
     }
     for (int k = 0; k < Staging::kSlots; ++k) {
@@ -1317,7 +1462,7 @@ void h2tap_close(h2tap_engine *e) {
     cudaFreeHost(e->small_host);
     e->published.reset();
     e->accepted.reset();
-    for (auto &t : e->tables) for (auto &c : t.col) { c.cur.reset(); c.spare.reset(); }
+    for (auto &t : e->tables) for (auto &c : t.col) { c.cur.reset(); c.alt.reset(); c.bits.reset(); }
     e->arena.bufs.clear();
     e->load_arena.bufs.clear();
     cudaStreamDestroy(e->compute);

@@ -194,6 +194,13 @@ void launch_q18_permute(const Q18Row *rows, const long long *amt, const unsigned
 void launch_stats_init(int *out, int n_pairs, cudaStream_t st);
 void launch_gate(unsigned long long ns, cudaStream_t st);  // profiling only  // pairs of (INT_MAX, INT_MIN)
 void launch_minmax_i32(const int32_t *p, uint64_t n, int *out, int num_sms, cudaStream_t st);
+// copy-on-write of updated columns (NEXT-1): page = kCowPageRows rows, one dirty bit per page
+constexpr uint64_t kCowPageRows = 4096;
+void launch_cow_catchup(void *dst, const void *src, uint32_t es, const uint32_t *bits,
+                        uint64_t synced_rows, uint64_t n_rows, unsigned long long *pages_copied,
+                        int num_sms, cudaStream_t st);
+void launch_apply_updates(void *col, uint32_t es, uint32_t *bits, const uint32_t *rows,
+                          const void *vals, uint64_t n, int num_sms, cudaStream_t st);
 
 // ---------------------------------------------------------------- helpers --
 // Every launcher counts the kernels it launches (reported per query as kernel_launches).

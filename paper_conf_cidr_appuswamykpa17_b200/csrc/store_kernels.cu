@@ -3,6 +3,14 @@
 // The planner uses them to lay out join indexes; they are metadata of the
 // snapshot, exactly like its row counts, and are published atomically with the epoch.
 // (Refresh-side kernels are not counted in a query's kernel_launches.)
+//
+// In-place updates (the paper's copy-on-write): a
+// column that receives updates keeps two device buffers, the visible version `cur` and a shadow
+// `alt` (the previous version). A one-bit-per-page map records the pages where the two differ.
+// A new version is built in the shadow: cow_catchup copies the dirty pages (and the rows
+// appended since the shadow was last in sync) cur -> alt, apply_updates scatters the new values
+// into alt and marks their pages; then the engine swaps the roles. Views of earlier epochs keep
+// reading their own buffer; page-granular traffic replaces a whole-column copy per epoch.
 #include <climits>
 #include <cstdint>
 #include <cuda_runtime.h>
@@ -45,7 +53,72 @@ __global__ void gate_kernel(unsigned long long ns) {
     } while (t - t0 < ns);
 }
 
+// Copy, cur -> alt, every page whose dirty bit is set among pages [0, synced_pages) and every
+// page overlapping rows [tail_lo, n_rows). One block per page at a time (grid-stride over pages);
+// 16-byte vectors, byte ranges rounded up to 16 (buffers carry >= kPadRows rows of padding).
+__global__ void __launch_bounds__(256) cow_catchup_kernel(uint8_t *__restrict__ dst,
+                                                          const uint8_t *__restrict__ src,
+                                                          uint32_t es, const uint32_t *__restrict__ bits,
+                                                          uint64_t synced_rows, uint64_t n_rows,
+                                                          unsigned long long *pages_copied) {
+    const uint64_t npages = (n_rows + kCowPageRows - 1) / kCowPageRows;
+    const uint64_t tail_page = synced_rows / kCowPageRows;
+    for (uint64_t p = blockIdx.x; p < npages; p += gridDim.x) {
+        const bool dirty = p >= tail_page || ((__ldg(bits + (p >> 5)) >> (p & 31)) & 1u);
+        if (!dirty) continue;
+        const uint64_t lo = p * kCowPageRows * es;
+        const uint64_t row_hi = (p + 1) * kCowPageRows < n_rows ? (p + 1) * kCowPageRows : n_rows;
+        const uint64_t hi = (row_hi * es + 15) & ~15ull;
+        const uint4 *s4 = reinterpret_cast<const uint4 *>(src + lo);
+        uint4 *d4 = reinterpret_cast<uint4 *>(dst + lo);
+        const uint64_t nv = (hi - lo) / 16;
+        for (uint64_t i = threadIdx.x; i < nv; i += blockDim.x) __stcs(d4 + i, __ldcs(s4 + i));
+        if (threadIdx.x == 0) atomicAdd(pages_copied, 1ull);
+    }
+}
+
+// alt[rows[i]] = vals[i], and mark the page of rows[i] dirty (cur and alt now differ there).
+// The bit is read first so a page hit by many updates costs one atomic, not one per row.
+template <class T>
+__global__ void __launch_bounds__(256) apply_updates_kernel(T *__restrict__ col, uint32_t *bits,
+                                                            const uint32_t *__restrict__ rows,
+                                                            const T *__restrict__ vals, uint64_t n) {
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
+        const uint32_t r = __ldg(rows + i);
+        col[r] = __ldg(vals + i);
+        const uint32_t page = r / kCowPageRows;
+        const uint32_t m = 1u << (page & 31);
+        if (!(__ldcg(bits + (page >> 5)) & m)) atomicOr(bits + (page >> 5), m);
+    }
+}
+
 }  // namespace
+
+void launch_cow_catchup(void *dst, const void *src, uint32_t es, const uint32_t *bits,
+                        uint64_t synced_rows, uint64_t n_rows, unsigned long long *pages_copied,
+                        int num_sms, cudaStream_t st) {
+    if (!n_rows) return;
+    const uint64_t npages = (n_rows + kCowPageRows - 1) / kCowPageRows;
+    const uint64_t cap = (uint64_t)num_sms * 8;
+    cow_catchup_kernel<<<(unsigned)(npages < cap ? npages : cap), 256, 0, st>>>(
+        static_cast<uint8_t *>(dst), static_cast<const uint8_t *>(src), es, bits, synced_rows, n_rows,
+        pages_copied);
+}
+
+void launch_apply_updates(void *col, uint32_t es, uint32_t *bits, const uint32_t *rows,
+                          const void *vals, uint64_t n, int num_sms, cudaStream_t st) {
+    if (!n) return;
+    uint64_t blocks = (n + 255) / 256;
+    const uint64_t cap = (uint64_t)num_sms * 8;
+    if (blocks > cap) blocks = cap;
+    if (es == 4)
+        apply_updates_kernel<int32_t><<<(unsigned)blocks, 256, 0, st>>>(
+            static_cast<int32_t *>(col), bits, rows, static_cast<const int32_t *>(vals), n);
+    else
+        apply_updates_kernel<int64_t><<<(unsigned)blocks, 256, 0, st>>>(
+            static_cast<int64_t *>(col), bits, rows, static_cast<const int64_t *>(vals), n);
+}
 
 void launch_gate(unsigned long long ns, cudaStream_t st) { gate_kernel<<<1, 1, 0, st>>>(ns); }
 

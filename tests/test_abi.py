@@ -35,7 +35,10 @@ def test_struct_layouts_match_header(h, tmp_path):
     import ctypes as C
     import subprocess
     structs = {"h2tap_column": h.h2tap_column, "h2tap_table": h.h2tap_table,
-               "h2tap_config": h.h2tap_config, "h2tap_result": h.h2tap_result}
+               "h2tap_config": h.h2tap_config, "h2tap_result": h.h2tap_result,
+               "h2tap_field": h.h2tap_field, "h2tap_row_table": h.h2tap_row_table,
+               "h2tap_query": h.h2tap_query, "h2tap_update": h.h2tap_update,
+               "h2tap_store_stats": h.h2tap_store_stats}
     lines = ['#include <stdio.h>', '#include <stddef.h>', '#include "h2tap.h"', 'int main(void){']
     for name, cls in structs.items():
         lines.append(f'printf("{name} %zu\\n", sizeof({name}));')
@@ -75,6 +78,9 @@ def test_bad_calls_fail_cleanly_without_gpu(h):
     assert h._lib.h2tap_run_query(None, 6, None, 0, None) == h.H2TAP_EINVAL
     assert h._lib.h2tap_load_snapshot(None, None, 0, 1) == h.H2TAP_EINVAL
     assert h._lib.h2tap_open(None, None) == h.H2TAP_EINVAL
+    assert h._lib.h2tap_refresh(None, None, 0, None, 0, 1, 0) == h.H2TAP_EINVAL
+    assert h._lib.h2tap_refresh_rows(None, None, 0, None, 0, 1, 0) == h.H2TAP_EINVAL
+    assert h._lib.h2tap_get_store_stats(None, None) == h.H2TAP_EINVAL
     h._lib.h2tap_free(None)
     h._lib.h2tap_close(None)
 
