@@ -88,7 +88,7 @@ class h2tap_store_stats(C.Structure):
                 ("rows_appended", C.c_uint64), ("rows_updated", C.c_uint64),
                 ("cow_pages_copied", C.c_uint64), ("cow_full_copies", C.c_uint64),
                 ("device_bytes", C.c_uint64), ("last_load_ms", C.c_double),
-                ("last_update_ms", C.c_double)]
+                ("last_update_h2d_ms", C.c_double), ("last_update_ms", C.c_double)]
 
 
 class h2tap_config(C.Structure):

@@ -210,8 +210,9 @@ using ViewP = std::shared_ptr<const View>;
 struct ColState {
     // cur: the latest accepted version. alt: the shadow (an earlier version, or a spare for full
     // reloads); when alt_valid, alt equals cur on rows [0, alt_synced) except on the pages whose
-    // bit is set in `bits` (copy-on-write of in-place updates, store_kernels.cu)
-    DevBufP cur, alt, bits;
+    // bit is set in `bits` (copy-on-write of in-place updates, store_kernels.cu); bits_next is
+    // the map the next update fills
+    DevBufP cur, alt, bits, bits_next;
     uint64_t cap_rows = 0;
     bool alt_valid = false;
     uint64_t alt_synced = 0;
@@ -227,7 +228,8 @@ struct Pending {
     uint64_t epoch;
     std::shared_ptr<View> view;   // becomes visible (const) at publish
     cudaEvent_t done;
-    cudaEvent_t t0, t1, t2;       // timing: begin, loads done, updates done (copy stream)
+    cudaEvent_t t0, t1, t2, t3;   // timing (copy stream): begin, loads done, update arrays
+                                  // uploaded, updates applied
     bool loaded[kTables], full[kTables], updated[kTables];
     int *stats_host;              // pinned [kTables][kStatCols][2] delta min/max, then the u64
                                   // count of pages copied into shadows (kStatBytes offset)
@@ -294,6 +296,9 @@ struct h2tap_engine {
     // the Q18 probe keeps register prefetch at high occupancy — its dependent lookups and atomics
     // need more warps than a one-block-per-SM shared-memory ring leaves (H2TAP_PROBE=tma: ring)
     bool scan_tma = true, probe_tma = false;
+    // in-place updates copy only the dirty pages into the shadow (H2TAP_COW=full: always copy the
+    // whole column — the A/B baseline of scripts/cow_bench.py)
+    bool cow_full = false;
     ncclComm_t comm = nullptr;
     cudaStream_t compute = nullptr, copy = nullptr;
     cudaEvent_t q_begin = nullptr, q_end = nullptr;
@@ -359,17 +364,21 @@ void publish_ready(h2tap_engine *e, bool wait) {
             CK(cudaEventElapsedTime(&a, p.t0, p.t1));
             CK(cudaEventElapsedTime(&b, p.t1, p.t2));
             S.last_load_ms = a;
+            S.last_update_h2d_ms = b;
+            CK(cudaEventElapsedTime(&b, p.t2, p.t3));
             S.last_update_ms = b;
         }
         {
             std::lock_guard<std::mutex> gv(e->view_mu);
             e->published = p.view;
         }
-        for (cudaEvent_t ev : {p.done, p.t0, p.t1, p.t2}) cudaEventDestroy(ev);
+        for (cudaEvent_t ev : {p.done, p.t0, p.t1, p.t2, p.t3}) cudaEventDestroy(ev);
         e->host_pool->put(p.stats_block.first, p.stats_block.second);
         e->pending.pop_front();
     }
 }
+
+inline size_t round_up16(size_t b) { return (b + 15) & ~size_t(15); }
 
 bool host_is_pinned(const void *p) {
     cudaPointerAttributes a;
@@ -379,6 +388,28 @@ bool host_is_pinned(const void *p) {
     }
     return a.type == cudaMemoryTypeHost;
 }
+
+// The next slot of the pinned staging ring, once its previous DMA has drained; staging_dma
+// sends its first `bytes` to `dst` on the copy stream (the engine owns the bytes: no wait).
+void *staging_slot(h2tap_engine *e) {
+    Staging &S = e->staging;
+    const int k = S.next;
+    if (!S.buf[k]) {
+        CK(cudaMallocHost(&S.buf[k], Staging::kChunk));
+        CK(cudaEventCreateWithFlags(&S.ev[k], cudaEventDisableTiming));
+    } else {
+        CK(cudaEventSynchronize(S.ev[k]));
+    }
+    return S.buf[k];
+}
+void staging_dma(h2tap_engine *e, void *dst, size_t bytes) {
+    Staging &S = e->staging;
+    const int k = S.next;
+    S.next = (S.next + 1) % Staging::kSlots;
+    CK(cudaMemcpyAsync(dst, S.buf[k], bytes, cudaMemcpyHostToDevice, e->copy));
+    CK(cudaEventRecord(S.ev[k], e->copy));
+}
+constexpr size_t kPackUpdateBytes = 256u << 10;
 
 // Copy `bytes` from host `src` to device `dst` on the copy stream. Pinned sources are DMA'd
 // directly (returns true: the caller must wait before returning); pageable ones go through the
@@ -500,7 +531,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
     pend.stats_host = static_cast<int *>(pend.stats_block.first);
     int *stats_dev = static_cast<int *>(e->load_arena.get("load.stats", kStatBytes + 8));
     auto *pages_dev = reinterpret_cast<unsigned long long *>(reinterpret_cast<char *>(stats_dev) + kStatBytes);
-    for (cudaEvent_t *ev : {&pend.t0, &pend.t1, &pend.t2}) CK(cudaEventCreate(ev));
+    for (cudaEvent_t *ev : {&pend.t0, &pend.t1, &pend.t2, &pend.t3}) CK(cudaEventCreate(ev));
     CK(cudaEventRecord(pend.t0, e->copy));
     launch_stats_init(stats_dev, kTables * kStatCols, e->copy);
     CK(cudaMemsetAsync(pages_dev, 0, 8, e->copy));
@@ -571,7 +602,30 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
                                       stats_dev + (t.table_id * kStatCols + c) * 2, e->num_sms, e->copy);
     }
     CK(cudaEventRecord(pend.t1, e->copy));
-    // ---- in-place updates: rebuild each updated column in its shadow buffer (copy-on-write)
+    // ---- in-place updates: upload every update's row ids and values first (one arena region;
+    // the device-side phase below then runs without waiting on the host), then rebuild each
+    // updated column in its shadow buffer (copy-on-write)
+    std::vector<size_t> upd_off(nupdates + 1, 0);
+    for (uint32_t i = 0; i < nupdates; ++i)
+        upd_off[i + 1] = upd_off[i] + round_up16(updates[i].n * 4) + round_up16(updates[i].n * type_size(updates[i].type));
+    char *upd_dev = nupdates ? static_cast<char *>(e->load_arena.get("upd.arrays", upd_off[nupdates] + 16)) : nullptr;
+    if (nupdates && upd_off[nupdates] <= kPackUpdateBytes) {
+        // small update sets are latency-bound: pack them into one staging slot, one DMA
+        char *stage = static_cast<char *>(staging_slot(e));
+        for (uint32_t i = 0; i < nupdates; ++i) {
+            const h2tap_update &u = updates[i];
+            if (u.n) std::memcpy(stage + upd_off[i], u.row_ids, u.n * 4);
+            if (u.n) std::memcpy(stage + upd_off[i] + round_up16(u.n * 4), u.values, u.n * type_size(u.type));
+        }
+        staging_dma(e, upd_dev, upd_off[nupdates]);
+    } else {
+        for (uint32_t i = 0; i < nupdates; ++i) {
+            const h2tap_update &u = updates[i];
+            must_wait |= h2d(e, upd_dev + upd_off[i], u.row_ids, u.n * 4);
+            must_wait |= h2d(e, upd_dev + upd_off[i] + round_up16(u.n * 4), u.values, u.n * type_size(u.type));
+        }
+    }
+    CK(cudaEventRecord(pend.t2, e->copy));
     for (uint32_t i = 0; i < nupdates; ++i) {
         const h2tap_update &u = updates[i];
         ColState &cs = e->tables[u.table_id].col[u.column_id];
@@ -580,30 +634,30 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         const uint64_t words = (cs.cap_rows + kCowPageRows * 32 - 1) / (kCowPageRows * 32);
         if (!cs.bits || cs.bits->bytes < words * 4) {
             cs.bits = dev_alloc(words * 4, e->device);
+            cs.bits_next = dev_alloc(words * 4, e->device);
             cs.alt_valid = false;  // no record of where alt differs
         }
-        uint32_t *bits = static_cast<uint32_t *>(cs.bits->ptr);
+        uint32_t *next_bits = static_cast<uint32_t *>(cs.bits_next->ptr);
         const bool reuse = cs.alt && cs.alt.use_count() == 1 && cs.alt->bytes >= cs.cap_rows * es;
-        if (reuse && cs.alt_valid) {
-            launch_cow_catchup(cs.alt->ptr, cs.cur->ptr, (uint32_t)es, bits, cs.alt_synced, n_rows,
-                               pages_dev, e->num_sms, e->copy);
+        if (reuse && cs.alt_valid && !e->cow_full) {
+            launch_cow_catchup(cs.alt->ptr, cs.cur->ptr, (uint32_t)es, static_cast<const uint32_t *>(cs.bits->ptr),
+                               next_bits, words, cs.alt_synced, n_rows, pages_dev, e->num_sms, e->copy);
         } else {
             if (!reuse) cs.alt = dev_alloc(cs.cap_rows * es, e->device);
             if (n_rows) CK(cudaMemcpyAsync(cs.alt->ptr, cs.cur->ptr, n_rows * es, cudaMemcpyDeviceToDevice, e->copy));
+            CK(cudaMemsetAsync(next_bits, 0, words * 4, e->copy));
             pend.full_copies += 1;
         }
-        CK(cudaMemsetAsync(bits, 0, words * 4, e->copy));
         if (u.n) {
-            auto *rows_d = static_cast<uint32_t *>(e->load_arena.get("upd.rows", u.n * 4));
-            void *vals_d = e->load_arena.get("upd.vals", u.n * es);
-            must_wait |= h2d(e, rows_d, u.row_ids, u.n * 4);
-            must_wait |= h2d(e, vals_d, u.values, u.n * es);
-            launch_apply_updates(cs.alt->ptr, (uint32_t)es, bits, rows_d, vals_d, u.n, e->num_sms, e->copy);
+            const auto *rows_d = reinterpret_cast<const uint32_t *>(upd_dev + upd_off[i]);
+            const void *vals_d = upd_dev + upd_off[i] + round_up16(u.n * 4);
+            launch_apply_updates(cs.alt->ptr, (uint32_t)es, next_bits, rows_d, vals_d, u.n, e->num_sms, e->copy);
             if (u.table_id != H2TAP_T_ITEM && u.column_id < (uint32_t)kStatCols)  // zone map: widen
                 launch_minmax_i32(static_cast<const int32_t *>(vals_d), u.n,
                                   stats_dev + (u.table_id * kStatCols + u.column_id) * 2, e->num_sms, e->copy);
         }
         std::swap(cs.cur, cs.alt);
+        std::swap(cs.bits, cs.bits_next);
         cs.alt_valid = true;
         cs.alt_synced = n_rows;
         v->col[u.table_id][u.column_id] = cs.cur->ptr;
@@ -611,7 +665,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         pend.updated[u.table_id] = true;
         pend.rows_updated += u.n;
     }
-    CK(cudaEventRecord(pend.t2, e->copy));
+    CK(cudaEventRecord(pend.t3, e->copy));
     CK(cudaGetLastError());
     CK(cudaMemcpyAsync(pend.stats_host, stats_dev, kStatBytes + 8, cudaMemcpyDeviceToHost, e->copy));
     CK(cudaEventCreateWithFlags(&pend.done, cudaEventDisableTiming));
@@ -1264,6 +1318,7 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         e->num_sms = prop.multiProcessorCount;
         if (const char *impl = std::getenv("H2TAP_SCAN")) e->scan_tma = std::strcmp(impl, "ldg") != 0;
         if (const char *impl = std::getenv("H2TAP_PROBE")) e->probe_tma = std::strcmp(impl, "tma") == 0;
+        if (const char *impl = std::getenv("H2TAP_COW")) e->cow_full = std::strcmp(impl, "full") == 0;
 
         CK(cudaStreamCreateWithFlags(&e->compute, cudaStreamNonBlocking));
         CK(cudaStreamCreateWithFlags(&e->copy, cudaStreamNonBlocking));
@@ -1335,7 +1390,7 @@ h2tap_status h2tap_get_store_stats(h2tap_engine *e, h2tap_store_stats *out) {
         uint64_t bytes = 0;
         for (auto &t : e->tables)
             for (auto &c : t.col)
-                for (const DevBufP *b : {&c.cur, &c.alt, &c.bits})
+                for (const DevBufP *b : {&c.cur, &c.alt, &c.bits, &c.bits_next})
                     if (*b) bytes += (*b)->bytes;
         out->device_bytes = bytes;
         return H2TAP_OK;
@@ -1449,7 +1504,7 @@ void h2tap_close(h2tap_engine *e) {
     cudaStreamSynchronize(e->copy);
     if (e->comm) ncclCommDestroy(e->comm);
     for (auto &p : e->pending) {
-        for (cudaEvent_t ev : {p.done, p.t0, p.t1, p.t2}) cudaEventDestroy(ev);
+        for (cudaEvent_t ev : {p.done, p.t0, p.t1, p.t2, p.t3}) cudaEventDestroy(ev);
         e->host_pool->put(p.stats_block.first, p.stats_block.second);
     }
     for (int k = 0; k < Staging::kSlots; ++k) {
@@ -1462,7 +1517,7 @@ void h2tap_close(h2tap_engine *e) {
     cudaFreeHost(e->small_host);
     e->published.reset();
     e->accepted.reset();
-    for (auto &t : e->tables) for (auto &c : t.col) { c.cur.reset(); c.alt.reset(); c.bits.reset(); }
+    for (auto &t : e->tables) for (auto &c : t.col) { c.cur.reset(); c.alt.reset(); c.bits.reset(); c.bits_next.reset(); }
     e->arena.bufs.clear();
     e->load_arena.bufs.clear();
     cudaStreamDestroy(e->compute);

@@ -196,9 +196,11 @@ void launch_gate(unsigned long long ns, cudaStream_t st);  // profiling only  //
 void launch_minmax_i32(const int32_t *p, uint64_t n, int *out, int num_sms, cudaStream_t st);
 // copy-on-write of updated columns (NEXT-1): page = kCowPageRows rows, one dirty bit per page
 constexpr uint64_t kCowPageRows = 4096;
+static_assert(kCowPageRows * 4 == 4 * 16 * 256, "catch-up kernel: one page = 4/8 uint4 per thread");
+// copy dirty pages (bits) and rows [synced_rows, n_rows) cur -> alt; clear next_bits[0, nwords)
 void launch_cow_catchup(void *dst, const void *src, uint32_t es, const uint32_t *bits,
-                        uint64_t synced_rows, uint64_t n_rows, unsigned long long *pages_copied,
-                        int num_sms, cudaStream_t st);
+                        uint32_t *next_bits, uint64_t nwords, uint64_t synced_rows, uint64_t n_rows,
+                        unsigned long long *pages_copied, int num_sms, cudaStream_t st);
 void launch_apply_updates(void *col, uint32_t es, uint32_t *bits, const uint32_t *rows,
                           const void *vals, uint64_t n, int num_sms, cudaStream_t st);
 

@@ -55,55 +55,88 @@ __global__ void gate_kernel(unsigned long long ns) {
 
 // Copy, cur -> alt, every page whose dirty bit is set among pages [0, synced_pages) and every
 // page overlapping rows [tail_lo, n_rows). One block per page at a time (grid-stride over pages);
-// 16-byte vectors, byte ranges rounded up to 16 (buffers carry >= kPadRows rows of padding).
+// a full page is moved with every load of a thread issued before its stores (16 KB / 32 KB in
+// flight per block); byte ranges rounded up to 16 (buffers carry >= kPadRows rows of padding).
+// The same launch clears `next_bits`, the map apply_updates fills for the next epoch.
+template <int kVecPerThread>  // = kCowPageRows * es / 16 / 256: 4 (int32) or 8 (int64)
 __global__ void __launch_bounds__(256) cow_catchup_kernel(uint8_t *__restrict__ dst,
                                                           const uint8_t *__restrict__ src,
-                                                          uint32_t es, const uint32_t *__restrict__ bits,
+                                                          const uint32_t *__restrict__ bits,
+                                                          uint32_t *__restrict__ next_bits, uint64_t nwords,
                                                           uint64_t synced_rows, uint64_t n_rows,
                                                           unsigned long long *pages_copied) {
+    constexpr uint64_t kPageBytes = (uint64_t)kVecPerThread * 16 * 256;
+    for (uint64_t w = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; w < nwords;
+         w += (uint64_t)gridDim.x * blockDim.x)
+        next_bits[w] = 0u;
     const uint64_t npages = (n_rows + kCowPageRows - 1) / kCowPageRows;
     const uint64_t tail_page = synced_rows / kCowPageRows;
+    const uint64_t row_bytes = kPageBytes / kCowPageRows;
     for (uint64_t p = blockIdx.x; p < npages; p += gridDim.x) {
         const bool dirty = p >= tail_page || ((__ldg(bits + (p >> 5)) >> (p & 31)) & 1u);
         if (!dirty) continue;
-        const uint64_t lo = p * kCowPageRows * es;
-        const uint64_t row_hi = (p + 1) * kCowPageRows < n_rows ? (p + 1) * kCowPageRows : n_rows;
-        const uint64_t hi = (row_hi * es + 15) & ~15ull;
-        const uint4 *s4 = reinterpret_cast<const uint4 *>(src + lo);
-        uint4 *d4 = reinterpret_cast<uint4 *>(dst + lo);
-        const uint64_t nv = (hi - lo) / 16;
-        for (uint64_t i = threadIdx.x; i < nv; i += blockDim.x) __stcs(d4 + i, __ldcs(s4 + i));
+        const uint4 *s4 = reinterpret_cast<const uint4 *>(src + p * kPageBytes);
+        uint4 *d4 = reinterpret_cast<uint4 *>(dst + p * kPageBytes);
+        if ((p + 1) * kCowPageRows <= n_rows) {
+            uint4 v[kVecPerThread];
+#pragma unroll
+            for (int k = 0; k < kVecPerThread; ++k) v[k] = __ldcs(s4 + k * 256 + threadIdx.x);
+#pragma unroll
+            for (int k = 0; k < kVecPerThread; ++k) __stcs(d4 + k * 256 + threadIdx.x, v[k]);
+        } else {  // ragged last page
+            const uint64_t nv = ((n_rows - p * kCowPageRows) * row_bytes + 15) / 16;
+            for (uint64_t i = threadIdx.x; i < nv; i += blockDim.x) __stcs(d4 + i, __ldcs(s4 + i));
+        }
         if (threadIdx.x == 0) atomicAdd(pages_copied, 1ull);
     }
 }
 
 // alt[rows[i]] = vals[i], and mark the page of rows[i] dirty (cur and alt now differ there).
-// The bit is read first so a page hit by many updates costs one atomic, not one per row.
+// Updates arrive clustered (a delivered order's lines are adjacent rows): a lane whose page
+// equals its left neighbour's leaves the bit to that lane, and the word is read first, so a page
+// costs about one atomic, not one per row.
 template <class T>
 __global__ void __launch_bounds__(256) apply_updates_kernel(T *__restrict__ col, uint32_t *bits,
                                                             const uint32_t *__restrict__ rows,
                                                             const T *__restrict__ vals, uint64_t n) {
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
-        const uint32_t r = __ldg(rows + i);
-        col[r] = __ldg(vals + i);
-        const uint32_t page = r / kCowPageRows;
+    const int lane = threadIdx.x & 31;
+    // every lane of a warp runs the same iterations (stride and start are warp-aligned)
+    for (uint64_t base = (uint64_t)blockIdx.x * blockDim.x; base < n; base += stride) {
+        const uint64_t i = base + threadIdx.x;
+        const bool valid = i < n;
+        uint32_t page = 0xffffffffu;
+        if (valid) {
+            const uint32_t r = __ldg(rows + i);
+            col[r] = __ldg(vals + i);
+            page = r / kCowPageRows;
+        }
+        const uint32_t left = __shfl_up_sync(0xffffffffu, page, 1);
         const uint32_t m = 1u << (page & 31);
-        if (!(__ldcg(bits + (page >> 5)) & m)) atomicOr(bits + (page >> 5), m);
+        if (valid && !(lane > 0 && left == page) && !(__ldcg(bits + (page >> 5)) & m))
+            atomicOr(bits + (page >> 5), m);
     }
 }
 
 }  // namespace
 
 void launch_cow_catchup(void *dst, const void *src, uint32_t es, const uint32_t *bits,
-                        uint64_t synced_rows, uint64_t n_rows, unsigned long long *pages_copied,
-                        int num_sms, cudaStream_t st) {
-    if (!n_rows) return;
+                        uint32_t *next_bits, uint64_t nwords, uint64_t synced_rows, uint64_t n_rows,
+                        unsigned long long *pages_copied, int num_sms, cudaStream_t st) {
     const uint64_t npages = (n_rows + kCowPageRows - 1) / kCowPageRows;
     const uint64_t cap = (uint64_t)num_sms * 8;
-    cow_catchup_kernel<<<(unsigned)(npages < cap ? npages : cap), 256, 0, st>>>(
-        static_cast<uint8_t *>(dst), static_cast<const uint8_t *>(src), es, bits, synced_rows, n_rows,
-        pages_copied);
+    uint64_t grid = npages < cap ? npages : cap;
+    const uint64_t wgrid = (nwords + 255) / 256;
+    if (grid < wgrid) grid = wgrid < cap ? wgrid : cap;
+    if (!grid) return;
+    auto *d = static_cast<uint8_t *>(dst);
+    const auto *s = static_cast<const uint8_t *>(src);
+    if (es == 4)
+        cow_catchup_kernel<4><<<(unsigned)grid, 256, 0, st>>>(d, s, bits, next_bits, nwords, synced_rows,
+                                                              n_rows, pages_copied);
+    else
+        cow_catchup_kernel<8><<<(unsigned)grid, 256, 0, st>>>(d, s, bits, next_bits, nwords, synced_rows,
+                                                              n_rows, pages_copied);
 }
 
 void launch_apply_updates(void *col, uint32_t es, uint32_t *bits, const uint32_t *rows,
