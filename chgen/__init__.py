@@ -18,7 +18,9 @@ and never defines the CH tables). Two modes (reading R9 / SURVEY B9):
 
 Encodings (R4-R6): ids int32; timestamps int64 µs
 since 1970-01-01 UTC with SQL NULL stored as INT64_MIN; money int64 cents;
-o_carrier_id NULL stored as -1; c_last an int32 dictionary code 0..999.
+o_carrier_id NULL stored as -1; c_last an int32 dictionary code 0..999; i_data the
+TPC-C string (bytes) plus ``i_data_p2`` = (byte0 << 8) | byte1, the device encoding of its
+first two characters (what CH Q14's ``LIKE 'PR%'`` needs; R29).
 
 Every warehouse w draws from its own stream ``Philox(key=[seed, w])`` (item
 uses w = 0), so any warehouse range [a, b) reproduces byte-identical rows to
@@ -37,6 +39,7 @@ __all__ = [
     "DAY_US", "ts_us", "generate", "generate_item", "neworder_delta",
     "warehouse_ranges", "concat_tables", "TABLE_COLUMNS", "NewOrderState", "neworder_batch",
     "ROW_DTYPES", "to_records", "DeliveryState", "delivery_inputs", "delivery_batch",
+    "i_data_prefix2",
 ]
 
 
@@ -63,7 +66,7 @@ TABLE_COLUMNS = {
                ("o_all_local", np.int32), ("o_entry_d", np.int64)],
     "customer": [("c_w_id", np.int32), ("c_d_id", np.int32), ("c_id", np.int32),
                  ("c_last", np.int32)],
-    "item": [("i_id", np.int32), ("i_price", np.int64)],
+    "item": [("i_id", np.int32), ("i_price", np.int64), ("i_data", "S50"), ("i_data_p2", np.int32)],
 }
 
 
@@ -161,11 +164,32 @@ def _warehouse(w: int, seed: int, mode: str, sc: Scale):
     return {"order_line": ol, "orders": orders, "customer": customer}
 
 
+ALNUM = np.frombuffer(b"abcdefghijklmnopqrstuvwxyzABCDEFGHIJKLMNOPQRSTUVWXYZ0123456789", np.uint8)
+
+
+def i_data_prefix2(i_data) -> np.ndarray:
+    """(byte0 << 8) | byte1 of each string (0 for a missing byte)."""
+    b = np.frombuffer(np.asarray(i_data, dtype="S50").tobytes(), np.uint8).reshape(-1, 50)
+    return ((b[:, 0].astype(np.int32) << 8) | b[:, 1].astype(np.int32)).astype(np.int32)
+
+
 def generate_item(seed: int = 1, scale: Scale = FULL):
-    """item table (replicated on every rank), stream key [seed, 0]."""
+    """item table (replicated on every rank), stream key [seed, 0]. i_data per TPC-C 4.3.3.1
+    [EXT]: random a-string of length U[26, 50] over [a-zA-Z0-9]; 10 % contain "ORIGINAL" at a
+    random position."""
     rng = _rng(seed, 0)
-    return {"i_id": np.arange(1, scale.items + 1, dtype=np.int32),
-            "i_price": rng.integers(100, 10_001, size=scale.items, dtype=np.int64)}
+    n = scale.items
+    price = rng.integers(100, 10_001, size=n, dtype=np.int64)
+    length = rng.integers(26, 51, size=n)
+    chars = ALNUM[rng.integers(0, len(ALNUM), size=(n, 50))]
+    orig = rng.random(n) < 0.10
+    pos = rng.integers(0, length - 8 + 1)
+    for i in np.flatnonzero(orig):
+        chars[i, pos[i]:pos[i] + 8] = np.frombuffer(b"ORIGINAL", np.uint8)
+    chars[np.arange(50)[None, :] >= length[:, None]] = 0
+    i_data = chars.view("S50").reshape(n)
+    return {"i_id": np.arange(1, n + 1, dtype=np.int32), "i_price": price,
+            "i_data": i_data, "i_data_p2": i_data_prefix2(i_data)}
 
 
 def concat_tables(parts):

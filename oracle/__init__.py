@@ -1,4 +1,4 @@
-"""CPU oracle for CH-benCHmark Q1 / Q6 / Q18 — TEST INFRASTRUCTURE ONLY.
+"""CPU oracle for CH-benCHmark Q1 / Q6 / Q18 (and NEXT-2: Q14 / Q12 / Q4) — TEST INFRASTRUCTURE ONLY.
 
 Only ``tests/``, ``__graft_entry__.smoke()`` and ``bench.py`` (its ``cpu_baseline``
 leg and ``--impl reference``) may import this package. The product path
@@ -43,12 +43,17 @@ def build(force: bool = False) -> str:
 class _OL(C.Structure):
     _fields_ = [("n", C.c_int64), ("w_id", C.c_void_p), ("d_id", C.c_void_p), ("o_id", C.c_void_p),
                 ("number", C.c_void_p), ("delivery_d", C.c_void_p), ("quantity", C.c_void_p),
-                ("amount", C.c_void_p)]
+                ("amount", C.c_void_p), ("i_id", C.c_void_p)]
 
 
 class _O(C.Structure):
     _fields_ = [("n", C.c_int64), ("w_id", C.c_void_p), ("d_id", C.c_void_p), ("o_id", C.c_void_p),
-                ("c_id", C.c_void_p), ("ol_cnt", C.c_void_p), ("entry_d", C.c_void_p)]
+                ("c_id", C.c_void_p), ("ol_cnt", C.c_void_p), ("entry_d", C.c_void_p),
+                ("carrier_id", C.c_void_p)]
+
+
+class _I(C.Structure):
+    _fields_ = [("n", C.c_int64), ("i_id", C.c_void_p), ("i_data", C.c_void_p), ("width", C.c_int64)]
 
 
 class _C(C.Structure):
@@ -66,6 +71,9 @@ def _load():
         lib.oracle_q6.restype = C.c_int
         lib.oracle_q1.restype = C.c_int64
         lib.oracle_q18.restype = C.c_int64
+        lib.oracle_q14.restype = C.c_int
+        lib.oracle_q12.restype = C.c_int64
+        lib.oracle_q4.restype = C.c_int64
         _lib = lib
     return _lib
 
@@ -90,12 +98,23 @@ class _Keep:
         return _p(a)
 
 
+def _opt(t, name, dtype, keep):
+    return keep(_col(t, name, dtype)) if name in t else None
+
+
 def _ol_struct(ol, keep):
-    n = len(ol["ol_w_id"])
-    return _OL(n, keep(_col(ol, "ol_w_id", np.int32)), keep(_col(ol, "ol_d_id", np.int32)),
-               keep(_col(ol, "ol_o_id", np.int32)), keep(_col(ol, "ol_number", np.int32)),
-               keep(_col(ol, "ol_delivery_d", np.int64)), keep(_col(ol, "ol_quantity", np.int32)),
-               keep(_col(ol, "ol_amount", np.int64)))
+    n = len(ol["ol_w_id"]) if "ol_w_id" in ol else len(ol["ol_delivery_d"])
+    return _OL(n, _opt(ol, "ol_w_id", np.int32, keep), _opt(ol, "ol_d_id", np.int32, keep),
+               _opt(ol, "ol_o_id", np.int32, keep), _opt(ol, "ol_number", np.int32, keep),
+               keep(_col(ol, "ol_delivery_d", np.int64)), _opt(ol, "ol_quantity", np.int32, keep),
+               keep(_col(ol, "ol_amount", np.int64)), _opt(ol, "ol_i_id", np.int32, keep))
+
+
+def _o_struct(o, keep):
+    return _O(len(o["o_w_id"]), keep(_col(o, "o_w_id", np.int32)), keep(_col(o, "o_d_id", np.int32)),
+              keep(_col(o, "o_id", np.int32)), _opt(o, "o_c_id", np.int32, keep),
+              keep(_col(o, "o_ol_cnt", np.int32)), keep(_col(o, "o_entry_d", np.int64)),
+              _opt(o, "o_carrier_id", np.int32, keep))
 
 
 def _check(st):
@@ -143,9 +162,7 @@ def q18(tables, having):
     lib, keep = _load(), _Keep()
     ol = _ol_struct(tables["order_line"], keep)
     o, c = tables["orders"], tables["customer"]
-    os_ = _O(len(o["o_w_id"]), keep(_col(o, "o_w_id", np.int32)), keep(_col(o, "o_d_id", np.int32)),
-             keep(_col(o, "o_id", np.int32)), keep(_col(o, "o_c_id", np.int32)),
-             keep(_col(o, "o_ol_cnt", np.int32)), keep(_col(o, "o_entry_d", np.int64)))
+    os_ = _o_struct(o, keep)
     cs = _C(len(c["c_w_id"]), keep(_col(c, "c_w_id", np.int32)), keep(_col(c, "c_d_id", np.int32)),
             keep(_col(c, "c_id", np.int32)), keep(_col(c, "c_last", np.int32)))
     cap = max(1, len(o["o_w_id"]))
@@ -173,3 +190,51 @@ def apply_updates(tables, updates):
             col[np.asarray(rows, dtype=np.int64)] = values
             out[t][c] = col
     return out
+
+
+def q14(tables, d_lo, d_hi, prefix=b"PR"):
+    """CH Q14 (order_line ⋈ item): {"promo_revenue": float or None (NULL), "sum_promo",
+    "sum_amount", "count"} — promo_revenue = 100.0 * sum_promo / (100.0 + sum_amount) (cents)."""
+    lib, keep = _load(), _Keep()
+    ol = _ol_struct(tables["order_line"], keep)
+    it = tables["item"]
+    data = np.ascontiguousarray(np.asarray(it["i_data"], dtype="S50"))
+    its = _I(len(it["i_id"]), keep(_col(it, "i_id", np.int32)), keep(data), 50)
+    promo, isnull = C.c_double(), C.c_int32()
+    sp, sa, cnt = C.c_int64(), C.c_int64(), C.c_int64()
+    _check(lib.oracle_q14(C.byref(ol), C.byref(its), C.c_int64(d_lo), C.c_int64(d_hi),
+                          C.c_char_p(bytes(prefix)), C.byref(promo), C.byref(isnull), C.byref(sp),
+                          C.byref(sa), C.byref(cnt)))
+    return {"promo_revenue": None if isnull.value else promo.value, "sum_promo": sp.value,
+            "sum_amount": sa.value, "count": cnt.value}
+
+
+def _small_groups(fn, names, dtypes):
+    cap = 64
+    while True:
+        out = {k: np.zeros(cap, dt) for k, dt in zip(names, dtypes)}
+        n = fn(cap, *[_p(out[k]) for k in names])
+        _check(n if n < 0 else 0)
+        if n <= cap:
+            return {k: v[:n] for k, v in out.items()}
+        cap = n
+
+
+def q12(tables, d_hi):
+    """CH Q12 (orders ⋈ order_line): columns o_ol_cnt, high_line_count, low_line_count."""
+    lib, keep = _load(), _Keep()
+    ol = _ol_struct(tables["order_line"], keep)
+    o = _o_struct(tables["orders"], keep)
+    return _small_groups(lambda cap, *ps: lib.oracle_q12(C.byref(o), C.byref(ol), C.c_int64(d_hi),
+                                                         C.c_int64(cap), *ps),
+                         ["o_ol_cnt", "high_line_count", "low_line_count"], [np.int32, np.int64, np.int64])
+
+
+def q4(tables, e_lo, e_hi):
+    """CH Q4 (orders semi-join order_line): columns o_ol_cnt, order_count."""
+    lib, keep = _load(), _Keep()
+    ol = _ol_struct(tables["order_line"], keep)
+    o = _o_struct(tables["orders"], keep)
+    return _small_groups(lambda cap, *ps: lib.oracle_q4(C.byref(o), C.byref(ol), C.c_int64(e_lo),
+                                                        C.c_int64(e_hi), C.c_int64(cap), *ps),
+                         ["o_ol_cnt", "order_count"], [np.int32, np.int64])

@@ -284,3 +284,153 @@ done:
     map_free(&hc); map_free(&ho); map_free(&hg);
     return st == OR_OK ? ngroups : st;
 }
+
+/* ---------------------------------------------------------------- CH Q14 -- */
+/* i_data LIKE 'prefix%': case-sensitive prefix match of the NUL-padded fixed-width string. */
+static int like_prefix(const char *str, int64_t width, const char *prefix) {
+    int64_t i = 0;
+    for (; prefix[i]; i++)
+        if (i >= width || str[i] != prefix[i]) return 0;
+    return 1;
+}
+
+int oracle_q14(const or_order_line *ol, const or_item *it, int64_t d_lo, int64_t d_hi,
+               const char *prefix, double *promo_revenue, int32_t *is_null, int64_t *sum_promo,
+               int64_t *sum_amount, int64_t *count) {
+    ormap hi;
+    int st = OR_OK;
+    int64_t sp = 0, sa = 0, cnt = 0;
+    if (map_init(&hi, 1, it->n)) { st = OR_NOMEM; goto done; }
+    for (int64_t r = 0; r < it->n; r++) {                      /* join index on item (i_id) */
+        int64_t k[1] = {it->i_id[r]};
+        if (map_append(&hi, k, r) < 0) { st = OR_NOMEM; goto done; }
+    }
+    for (int64_t l = 0; l < ol->n; l++) {                      /* scan order_line */
+        sqlbool p = sql_and(ts_ge(ol->delivery_d[l], d_lo), ts_lt(ol->delivery_d[l], d_hi));
+        if (p != SQL_TRUE) continue;
+        int64_t k[1] = {ol->i_id[l]};
+        for (int64_t e = map_first(&hi, k); e >= 0; e = map_next_same(&hi, e, k)) {  /* ol_i_id = i_id */
+            int64_t irow = hi.val[e];
+            int64_t promo = like_prefix(it->i_data + irow * it->width, it->width, prefix) ? ol->amount[l] : 0;
+            if (__builtin_add_overflow(sp, promo, &sp) ||
+                __builtin_add_overflow(sa, ol->amount[l], &sa)) { st = OR_OVERFLOW; goto done; }
+            cnt++;
+        }
+    }
+    *is_null = cnt == 0;                                        /* SUM(empty) IS NULL -> NULL */
+    *promo_revenue = cnt ? (100.0 * (double)sp) / (100.0 + (double)sa) : 0.0;
+    *sum_promo = sp;
+    *sum_amount = sa;
+    *count = cnt;
+done:
+    map_free(&hi);
+    return st;
+}
+
+/* ------------------------------------------------------- Q12 / Q4 groups -- */
+typedef struct { int64_t key, a, b; } small_group;
+
+static int cmp_small(const void *x, const void *y) {
+    int64_t a = ((const small_group *)x)->key, b = ((const small_group *)y)->key;
+    return (a > b) - (a < b);
+}
+
+/* find-or-insert the group of `key` (GROUP BY o_ol_cnt) */
+static int64_t group_of(ormap *m, small_group **g, int64_t *n, int64_t *cap, int64_t key) {
+    int64_t k[1] = {key};
+    int64_t e = map_first(m, k);
+    if (e >= 0) return m->val[e];
+    if (*n == *cap) {
+        *cap *= 2;
+        small_group *ng = realloc(*g, sizeof(small_group) * *cap);
+        if (!ng) return OR_NOMEM;
+        *g = ng;
+    }
+    int64_t gi = (*n)++;
+    (*g)[gi].key = key; (*g)[gi].a = 0; (*g)[gi].b = 0;
+    if (map_append(m, k, gi) < 0) return OR_NOMEM;
+    return gi;
+}
+
+/* carrier = 1 OR carrier = 2 (NULL -> UNKNOWN); carrier <> 1 AND carrier <> 2 (NULL -> UNKNOWN) */
+static sqlbool carrier_eq(int32_t c, int32_t v) { return c == -1 ? SQL_UNKNOWN : (c == v ? SQL_TRUE : SQL_FALSE); }
+static sqlbool sql_or(sqlbool a, sqlbool b) {
+    if (a == SQL_TRUE || b == SQL_TRUE) return SQL_TRUE;
+    if (a == SQL_UNKNOWN || b == SQL_UNKNOWN) return SQL_UNKNOWN;
+    return SQL_FALSE;
+}
+static sqlbool sql_not(sqlbool a) { return a == SQL_UNKNOWN ? SQL_UNKNOWN : (a == SQL_TRUE ? SQL_FALSE : SQL_TRUE); }
+
+int64_t oracle_q12(const or_orders *o, const or_order_line *ol, int64_t d_hi, int64_t cap,
+                   int32_t *o_ol_cnt, int64_t *high_line_count, int64_t *low_line_count) {
+    ormap ho, hg;
+    int st = OR_OK;
+    int64_t ng = 0, gcap = 64;
+    small_group *g = malloc(sizeof(small_group) * gcap);
+    memset(&ho, 0, sizeof ho); memset(&hg, 0, sizeof hg);
+    if (!g || map_init(&ho, 3, o->n) || map_init(&hg, 1, 64)) { st = OR_NOMEM; goto done; }
+    for (int64_t r = 0; r < o->n; r++) {                       /* join index on orders */
+        int64_t k[3] = {o->w_id[r], o->d_id[r], o->o_id[r]};
+        if (map_append(&ho, k, r) < 0) { st = OR_NOMEM; goto done; }
+    }
+    for (int64_t l = 0; l < ol->n; l++) {                      /* scan order_line */
+        int64_t k[3] = {ol->w_id[l], ol->d_id[l], ol->o_id[l]};
+        for (int64_t e = map_first(&ho, k); e >= 0; e = map_next_same(&ho, e, k)) {
+            int64_t orow = ho.val[e];
+            /* o_entry_d <= ol_delivery_d AND ol_delivery_d < d_hi (NULL delivery -> UNKNOWN) */
+            sqlbool p = sql_and(sql_not(ts_lt(ol->delivery_d[l], o->entry_d[orow])),
+                                ts_lt(ol->delivery_d[l], d_hi));
+            if (p != SQL_TRUE) continue;
+            int64_t gi = group_of(&hg, &g, &ng, &gcap, o->ol_cnt[orow]);
+            if (gi < 0) { st = OR_NOMEM; goto done; }
+            int32_t c = o->carrier_id[orow];
+            if (sql_or(carrier_eq(c, 1), carrier_eq(c, 2)) == SQL_TRUE) g[gi].a++;
+            if (sql_and(sql_not(carrier_eq(c, 1)), sql_not(carrier_eq(c, 2))) == SQL_TRUE) g[gi].b++;
+        }
+    }
+    qsort(g, (size_t)ng, sizeof(small_group), cmp_small);       /* ORDER BY o_ol_cnt */
+    for (int64_t i = 0; i < ng && i < cap; i++) {
+        o_ol_cnt[i] = (int32_t)g[i].key;
+        high_line_count[i] = g[i].a;
+        low_line_count[i] = g[i].b;
+    }
+done:
+    free(g);
+    map_free(&ho); map_free(&hg);
+    return st == OR_OK ? ng : st;
+}
+
+int64_t oracle_q4(const or_orders *o, const or_order_line *ol, int64_t e_lo, int64_t e_hi,
+                  int64_t cap, int32_t *o_ol_cnt, int64_t *order_count) {
+    ormap hl, hg;
+    int st = OR_OK;
+    int64_t ng = 0, gcap = 64;
+    small_group *g = malloc(sizeof(small_group) * gcap);
+    memset(&hl, 0, sizeof hl); memset(&hg, 0, sizeof hg);
+    if (!g || map_init(&hl, 3, ol->n) || map_init(&hg, 1, 64)) { st = OR_NOMEM; goto done; }
+    for (int64_t l = 0; l < ol->n; l++) {                      /* index on order_line (w, d, o) */
+        int64_t k[3] = {ol->w_id[l], ol->d_id[l], ol->o_id[l]};
+        if (map_append(&hl, k, l) < 0) { st = OR_NOMEM; goto done; }
+    }
+    for (int64_t r = 0; r < o->n; r++) {                       /* scan orders */
+        /* o_entry_d >= e_lo AND o_entry_d < e_hi (entry is never NULL) */
+        if (!(o->entry_d[r] >= e_lo && o->entry_d[r] < e_hi)) continue;
+        int exists = 0;                                          /* EXISTS (correlated) */
+        int64_t k[3] = {o->w_id[r], o->d_id[r], o->o_id[r]};
+        for (int64_t e = map_first(&hl, k); e >= 0 && !exists; e = map_next_same(&hl, e, k))
+            exists = ts_ge(ol->delivery_d[hl.val[e]], o->entry_d[r]) == SQL_TRUE;
+        if (!exists) continue;
+        int64_t gi = group_of(&hg, &g, &ng, &gcap, o->ol_cnt[r]);
+        if (gi < 0) { st = OR_NOMEM; goto done; }
+        g[gi].a++;
+    }
+    qsort(g, (size_t)ng, sizeof(small_group), cmp_small);
+    for (int64_t i = 0; i < ng && i < cap; i++) {
+        o_ol_cnt[i] = (int32_t)g[i].key;
+        order_count[i] = g[i].a;
+    }
+done:
+    free(g);
+    map_free(&hl); map_free(&hg);
+    return st == OR_OK ? ng : st;
+}

@@ -5,7 +5,8 @@
  * legs may load liboracle.so. It shares no code, header, table or constant with the
  * CUDA path (paper_conf_cidr_appuswamykpa17_b200/, include/), and never includes them.
  *
- * What it computes: the plain SQL definitions of CH-benCHmark Q1, Q6 and Q18
+ * What it computes: the plain SQL definitions of CH-benCHmark Q1, Q6 and Q18, and (NEXT-2)
+ * Q14, Q12 and Q4
  * (SURVEY.md Appendix A.1 [EXT]; the paper's OLAP path is PAPER.md L524-572, its only
  * query text is "TPC-H Q6, a selection over the lineitem table", L687-688), evaluated
  * row at a time, single-threaded, with SQL three-valued logic for NULLs.
@@ -32,13 +33,22 @@ typedef struct {
     const int64_t *delivery_d;      /* INT64_MIN = NULL */
     const int32_t *quantity;
     const int64_t *amount;          /* cents */
+    const int32_t *i_id;            /* ol_i_id (Q14 only; may be NULL otherwise) */
 } or_order_line;
 
 typedef struct {
     int64_t n;
     const int32_t *w_id, *d_id, *o_id, *c_id, *ol_cnt;
     const int64_t *entry_d;
+    const int32_t *carrier_id;      /* -1 = NULL (Q12 only; may be NULL otherwise) */
 } or_orders;
+
+typedef struct {
+    int64_t n;
+    const int32_t *i_id;
+    const char *i_data;             /* n strings of `width` bytes each, NUL-padded */
+    int64_t width;
+} or_item;
 
 typedef struct {
     int64_t n;
@@ -74,6 +84,31 @@ int64_t oracle_q18(const or_customer *c, const or_orders *o, const or_order_line
                    int64_t having, int64_t cap,
                    int32_t *c_last, int32_t *c_id, int32_t *o_id, int64_t *o_entry_d,
                    int32_t *o_ol_cnt, int64_t *amount_sum, int32_t *o_w_id, int32_t *o_d_id);
+
+/* CH Q14: SELECT 100.00 * SUM(CASE WHEN i_data LIKE prefix || '%' THEN ol_amount ELSE 0 END)
+ *                / (1 + SUM(ol_amount)) AS promo_revenue
+ * FROM order_line, item WHERE ol_i_id = i_id AND ol_delivery_d >= d_lo AND ol_delivery_d < d_hi.
+ * Money in cents: promo_revenue = (100.0 * (double)sum_promo) / (100.0 + (double)sum_amount)
+ * (R30); NULL (*is_null = 1) when no joined row qualifies. LIKE is case-sensitive. */
+int oracle_q14(const or_order_line *ol, const or_item *it, int64_t d_lo, int64_t d_hi,
+               const char *prefix, double *promo_revenue, int32_t *is_null, int64_t *sum_promo,
+               int64_t *sum_amount, int64_t *count);
+
+/* CH Q12: SELECT o_ol_cnt,
+ *   SUM(CASE WHEN o_carrier_id = 1 OR o_carrier_id = 2 THEN 1 ELSE 0 END) AS high_line_count,
+ *   SUM(CASE WHEN o_carrier_id <> 1 AND o_carrier_id <> 2 THEN 1 ELSE 0 END) AS low_line_count
+ * FROM orders, order_line WHERE ol_w_id = o_w_id AND ol_d_id = o_d_id AND ol_o_id = o_id
+ *   AND o_entry_d <= ol_delivery_d AND ol_delivery_d < d_hi GROUP BY o_ol_cnt ORDER BY o_ol_cnt.
+ * Writes min(ngroups, cap) rows; returns ngroups or < 0. */
+int64_t oracle_q12(const or_orders *o, const or_order_line *ol, int64_t d_hi, int64_t cap,
+                   int32_t *o_ol_cnt, int64_t *high_line_count, int64_t *low_line_count);
+
+/* CH Q4: SELECT o_ol_cnt, COUNT(*) AS order_count FROM orders
+ * WHERE o_entry_d >= e_lo AND o_entry_d < e_hi AND EXISTS (SELECT * FROM order_line
+ *   WHERE o_id = ol_o_id AND o_w_id = ol_w_id AND o_d_id = ol_d_id AND ol_delivery_d >= o_entry_d)
+ * GROUP BY o_ol_cnt ORDER BY o_ol_cnt. Writes min(ngroups, cap) rows; returns ngroups or < 0. */
+int64_t oracle_q4(const or_orders *o, const or_order_line *ol, int64_t e_lo, int64_t e_hi,
+                  int64_t cap, int32_t *o_ol_cnt, int64_t *order_count);
 
 #ifdef __cplusplus
 }

@@ -41,15 +41,16 @@ def sqlite_load(tables):
     db = sqlite3.connect(":memory:")
     ol, o, c = tables["order_line"], tables["orders"], tables["customer"]
     db.execute("CREATE TABLE order_line (ol_w_id INT, ol_d_id INT, ol_o_id INT, ol_number INT,"
-               " ol_delivery_d INT, ol_quantity INT, ol_amount INT)")
+               " ol_delivery_d INT, ol_quantity INT, ol_amount INT, ol_i_id INT)")
     db.execute("CREATE TABLE orders (o_w_id INT, o_d_id INT, o_id INT, o_c_id INT, o_ol_cnt INT,"
                " o_entry_d INT, o_carrier_id INT)")
     db.execute("CREATE TABLE customer (c_w_id INT, c_d_id INT, c_id INT, c_last INT)")
     deliv = [None if int(v) == NULL_SENTINEL else int(v) for v in ol["ol_delivery_d"]]
-    db.executemany("INSERT INTO order_line VALUES (?,?,?,?,?,?,?)",
+    iid = ol["ol_i_id"].tolist() if "ol_i_id" in ol else [None] * len(deliv)
+    db.executemany("INSERT INTO order_line VALUES (?,?,?,?,?,?,?,?)",
                    zip(ol["ol_w_id"].tolist(), ol["ol_d_id"].tolist(), ol["ol_o_id"].tolist(),
                        ol["ol_number"].tolist(), deliv, ol["ol_quantity"].tolist(),
-                       ol["ol_amount"].tolist()))
+                       ol["ol_amount"].tolist(), iid))
     carrier = [None if int(v) == -1 else int(v) for v in o["o_carrier_id"]]
     db.executemany("INSERT INTO orders VALUES (?,?,?,?,?,?,?)",
                    zip(o["o_w_id"].tolist(), o["o_d_id"].tolist(), o["o_id"].tolist(),
@@ -60,6 +61,14 @@ def sqlite_load(tables):
                        c["c_last"].tolist()))
     db.execute("CREATE INDEX io ON orders (o_w_id, o_d_id, o_id)")
     db.execute("CREATE INDEX ic ON customer (c_w_id, c_d_id, c_id)")
+    db.execute("CREATE INDEX il ON order_line (ol_w_id, ol_d_id, ol_o_id)")
+    if "item" in tables and "i_data" in tables["item"]:
+        it = tables["item"]
+        db.execute("CREATE TABLE item (i_id INT, i_data TEXT)")
+        db.executemany("INSERT INTO item VALUES (?,?)",
+                       zip(it["i_id"].tolist(), [bytes(x).decode("latin-1") for x in it["i_data"]]))
+        db.execute("CREATE INDEX ii ON item (i_id)")
+    db.execute("PRAGMA case_sensitive_like = ON")  # SQL LIKE is case-sensitive
     return db
 
 
@@ -88,6 +97,34 @@ def sqlite_q18(db, having):
         "GROUP BY o_id, o_w_id, o_d_id, c_id, c_last, o_entry_d, o_ol_cnt "
         "HAVING SUM(ol_amount) > ? ORDER BY amount_sum DESC, o_entry_d",
         (having,)).fetchall()
+
+
+def sqlite_q14(db, d_lo, d_hi, prefix="PR"):
+    """CH Q14 verbatim, money converted to currency units per row (ol_amount / 100.0)."""
+    return db.execute(
+        "SELECT 100.00 * SUM(CASE WHEN i_data LIKE ? THEN ol_amount / 100.0 ELSE 0 END)"
+        " / (1 + SUM(ol_amount / 100.0)) AS promo_revenue,"
+        " SUM(CASE WHEN i_data LIKE ? THEN ol_amount ELSE 0 END), SUM(ol_amount), COUNT(*) "
+        "FROM order_line, item WHERE ol_i_id = i_id AND ol_delivery_d >= ? AND ol_delivery_d < ?",
+        (prefix + "%", prefix + "%", d_lo, d_hi)).fetchone()
+
+
+def sqlite_q12(db, d_hi):
+    return db.execute(
+        "SELECT o_ol_cnt,"
+        " SUM(CASE WHEN o_carrier_id = 1 OR o_carrier_id = 2 THEN 1 ELSE 0 END) AS high_line_count,"
+        " SUM(CASE WHEN o_carrier_id <> 1 AND o_carrier_id <> 2 THEN 1 ELSE 0 END) AS low_line_count "
+        "FROM orders, order_line WHERE ol_w_id = o_w_id AND ol_d_id = o_d_id AND ol_o_id = o_id"
+        " AND o_entry_d <= ol_delivery_d AND ol_delivery_d < ? GROUP BY o_ol_cnt ORDER BY o_ol_cnt",
+        (d_hi,)).fetchall()
+
+
+def sqlite_q4(db, e_lo, e_hi):
+    return db.execute(
+        "SELECT o_ol_cnt, COUNT(*) AS order_count FROM orders "
+        "WHERE o_entry_d >= ? AND o_entry_d < ? AND EXISTS (SELECT * FROM order_line"
+        " WHERE o_id = ol_o_id AND o_w_id = ol_w_id AND o_d_id = ol_d_id AND ol_delivery_d >= o_entry_d) "
+        "GROUP BY o_ol_cnt ORDER BY o_ol_cnt", (e_lo, e_hi)).fetchall()
 
 
 def sqlite_delivery(db, w, carrier, ts, districts):
@@ -161,6 +198,48 @@ def brute_q18(tables, having):
     return out
 
 
+def brute_q14(tables, d_lo, d_hi, prefix=b"PR"):
+    """(sum_promo, sum_amount, count) over the cartesian product order_line × item."""
+    L = _rows(tables["order_line"], ["ol_i_id", "ol_delivery_d", "ol_amount"])
+    items = list(zip(tables["item"]["i_id"].tolist(), [bytes(x) for x in tables["item"]["i_data"]]))
+    sp = sa = cnt = 0
+    for (iid, d, a), (i_id, data) in itertools.product(L, items):
+        d = _null(d)
+        if iid == i_id and d is not None and d_lo <= d < d_hi:
+            sp += a if data.startswith(prefix) else 0
+            sa += a
+            cnt += 1
+    return sp, sa, cnt
+
+
+def brute_q12(tables, d_hi):
+    O = _rows(tables["orders"], ["o_w_id", "o_d_id", "o_id", "o_ol_cnt", "o_carrier_id", "o_entry_d"])
+    L = _rows(tables["order_line"], ["ol_w_id", "ol_d_id", "ol_o_id", "ol_delivery_d"])
+    groups = {}
+    for (ow, od, oid, cnt, car, ent), (lw, ld, lo, d) in itertools.product(O, L):
+        d = _null(d)
+        if lw == ow and ld == od and lo == oid and d is not None and ent <= d and d < d_hi:
+            g = groups.setdefault(cnt, [0, 0])
+            if car != -1 and car in (1, 2):
+                g[0] += 1
+            if car != -1 and car not in (1, 2):
+                g[1] += 1
+    return [(k, g[0], g[1]) for k, g in sorted(groups.items())]
+
+
+def brute_q4(tables, e_lo, e_hi):
+    O = _rows(tables["orders"], ["o_w_id", "o_d_id", "o_id", "o_ol_cnt", "o_entry_d"])
+    L = _rows(tables["order_line"], ["ol_w_id", "ol_d_id", "ol_o_id", "ol_delivery_d"])
+    groups = {}
+    for (ow, od, oid, cnt, ent) in O:
+        if not (e_lo <= ent < e_hi):
+            continue
+        if any(lw == ow and ld == od and lo == oid and _null(d) is not None and d >= ent
+               for (lw, ld, lo, d) in L):
+            groups[cnt] = groups.get(cnt, 0) + 1
+    return sorted(groups.items())
+
+
 # ------------------------------------------------------------------- golden --
 def golden(name="tiny_ch.json"):
     with open(os.path.join(GOLDEN, name)) as f:
@@ -198,3 +277,43 @@ def table_rows(tables, t):
 def canon_rows(cols: dict, names):
     """Rows as a sorted list of tuples (canonical full-row sort for set comparison)."""
     return sorted(zip(*[np.asarray(cols[n]).tolist() for n in names]))
+
+
+def golden_next2(name="ch_next2.json"):
+    """The NEXT-2 fixture as generator-shaped tables (+ params and expected values)."""
+    with open(os.path.join(GOLDEN, name)) as f:
+        g = json.load(f)
+    ts_cols = ("ol_delivery_d", "o_entry_d")
+    i64_cols = ("ol_amount",)
+    tables = {}
+    for t in ("orders", "order_line"):
+        cols, rows = g[t]["columns"], g[t]["rows"]
+        tab = {}
+        for j, c in enumerate(cols):
+            vals = [r[j] for r in rows]
+            if c in ts_cols:
+                tab[c] = np.array([NULL_SENTINEL if v is None else iso_us(v) for v in vals], np.int64)
+            elif c in i64_cols:
+                tab[c] = np.array(vals, np.int64)
+            else:
+                tab[c] = np.array(vals, np.int32)
+        tables[t] = tab
+    ol = tables["order_line"]
+    n = len(ol["ol_w_id"])
+    ol["ol_number"] = ol.get("ol_number", np.ones(n, np.int32))
+    ol["ol_quantity"] = np.ones(n, np.int32)
+    ol["ol_supply_w_id"] = ol["ol_w_id"].copy()
+    o = tables["orders"]
+    o["o_all_local"] = np.ones(len(o["o_id"]), np.int32)
+    items = g["item"]["rows"]
+    data = np.array([s.encode() for _, s in items], dtype="S50")
+    b = np.frombuffer(data.tobytes(), np.uint8).reshape(-1, 50)
+    tables["item"] = {"i_id": np.array([i for i, _ in items], np.int32),
+                      "i_price": np.full(len(items), 100, np.int64), "i_data": data,
+                      "i_data_p2": ((b[:, 0].astype(np.int32) << 8) | b[:, 1]).astype(np.int32)}
+    tables["customer"] = {"c_w_id": np.zeros(0, np.int32), "c_d_id": np.zeros(0, np.int32),
+                          "c_id": np.zeros(0, np.int32), "c_last": np.zeros(0, np.int32)}
+    p = g["params"]
+    params = {"q14": (iso_us(p["q14"][0]), iso_us(p["q14"][1]), p["q14"][2].encode()),
+              "q12": (iso_us(p["q12"][0]),), "q4": (iso_us(p["q4"][0]), iso_us(p["q4"][1]))}
+    return tables, params, g["expected"]
