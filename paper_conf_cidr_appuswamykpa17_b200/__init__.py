@@ -35,6 +35,7 @@ STATUS_NAMES = {0: "OK", -1: "EINVAL", -2: "ESTALE", -3: "ENOMEM", -4: "ECUDA", 
 H2TAP_I32, H2TAP_I64, H2TAP_F64 = 1, 2, 3
 H2TAP_T_ORDER_LINE, H2TAP_T_ORDERS, H2TAP_T_CUSTOMER, H2TAP_T_ITEM = 1, 2, 3, 4
 H2TAP_Q1, H2TAP_Q6, H2TAP_Q18 = 1, 6, 18
+H2TAP_Q4, H2TAP_Q12, H2TAP_Q14 = 4, 12, 14  # NEXT-2 CH queries
 H2TAP_FULL_RELOAD = 1
 H2TAP_LOAD_ASYNC = 1
 H2TAP_RESULT_DEVICE = 1
@@ -55,7 +56,7 @@ SCHEMA = {
         ("o_entry_d", H2TAP_I64)]),
     "customer": (H2TAP_T_CUSTOMER, [
         ("c_w_id", H2TAP_I32), ("c_d_id", H2TAP_I32), ("c_id", H2TAP_I32), ("c_last", H2TAP_I32)]),
-    "item": (H2TAP_T_ITEM, [("i_id", H2TAP_I32), ("i_price", H2TAP_I64)]),
+    "item": (H2TAP_T_ITEM, [("i_id", H2TAP_I32), ("i_price", H2TAP_I64), ("i_data_p2", H2TAP_I32)]),
 }
 
 
@@ -469,9 +470,18 @@ def h2tap_c_last_name(code: int) -> str:
     return buf.value.decode()
 
 
+HOT_PATH_PLANS = (H2TAP_Q1, H2TAP_Q6, H2TAP_Q18)  # BASELINE north_star
+
+
 def plan_columns():
     """Columns each plan reads (what h2tap_load_snapshot must have provided)."""
     return {
+        H2TAP_Q14: {"order_line": ["ol_delivery_d", "ol_i_id", "ol_amount"],
+                    "item": ["i_id", "i_data_p2"]},
+        H2TAP_Q12: {"order_line": ["ol_w_id", "ol_d_id", "ol_o_id", "ol_delivery_d"],
+                    "orders": ["o_w_id", "o_d_id", "o_id", "o_ol_cnt", "o_carrier_id", "o_entry_d"]},
+        H2TAP_Q4: {"order_line": ["ol_w_id", "ol_d_id", "ol_o_id", "ol_delivery_d"],
+                   "orders": ["o_w_id", "o_d_id", "o_id", "o_ol_cnt", "o_entry_d"]},
         H2TAP_Q6: {"order_line": ["ol_delivery_d", "ol_quantity", "ol_amount"]},
         H2TAP_Q1: {"order_line": ["ol_number", "ol_delivery_d", "ol_quantity", "ol_amount"]},
         H2TAP_Q18: {"order_line": ["ol_w_id", "ol_d_id", "ol_o_id", "ol_amount"],
@@ -480,10 +490,11 @@ def plan_columns():
     }
 
 
-def hot_path_tables(tables: dict) -> dict:
-    """The subset of generated columns the hot path's plans read (union over Q1/Q6/Q18)."""
+def hot_path_tables(tables: dict, plans=HOT_PATH_PLANS) -> dict:
+    """The subset of generated columns that ``plans`` read (default: the hot path, Q1/Q6/Q18)."""
     want = {}
-    for spec in plan_columns().values():
+    spec_of = plan_columns()
+    for spec in (spec_of[p] for p in plans):
         for t, cols in spec.items():
             want.setdefault(t, [])
             for c in cols:

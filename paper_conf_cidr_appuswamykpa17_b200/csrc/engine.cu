@@ -83,13 +83,13 @@ struct Fail {  // thrown internally, converted to a status at the ABI boundary
 // ============================================================== schema ===
 constexpr int kTables = 5;  // index = table id (1..4)
 constexpr int kMaxCols = 9;
-const int kNcols[kTables] = {0, 9, 8, 4, 2};
+const int kNcols[kTables] = {0, 9, 8, 4, 3};
 const uint32_t kTypes[kTables][kMaxCols] = {
     {},
     {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64},
     {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64},
     {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32},
-    {H2TAP_I32, H2TAP_I64}};
+    {H2TAP_I32, H2TAP_I64, H2TAP_I32}};
 inline size_t type_size(uint32_t t) { return t == H2TAP_I32 ? 4 : 8; }
 constexpr uint64_t kPadRows = 64;  // over-allocation so 128-bit loads of the last tile stay in bounds
 
@@ -196,6 +196,8 @@ struct ResultImpl : h2tap_result {
 
 // =========================================================== snapshot ===
 constexpr int kStatCols = 3;  // min/max kept for the (w, d, id) key columns 0..2 of each table
+// (item: i_id only — its columns 1..2 are not keys)
+inline int stat_cols(int table) { return table == H2TAP_T_ITEM ? 1 : kStatCols; }
 struct View {  // immutable snapshot at one epoch (the paper's shallow-copied top container)
     uint64_t epoch = 0;
     uint64_t n[kTables] = {};
@@ -594,12 +596,11 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         pend.loaded[t.table_id] = true;
         pend.full[t.table_id] = full;
         // zone map of the appended rows' key columns, on the copy stream after their H2D
-        if (t.table_id != H2TAP_T_ITEM)
-            for (int c = 0; c < kStatCols; ++c)
-                if (v->col[t.table_id][c])
-                    launch_minmax_i32(static_cast<const int32_t *>(v->col[t.table_id][c]) + t.first_row,
-                                      t.row_count - t.first_row,
-                                      stats_dev + (t.table_id * kStatCols + c) * 2, e->num_sms, e->copy);
+        for (int c = 0; c < stat_cols(t.table_id); ++c)
+            if (v->col[t.table_id][c])
+                launch_minmax_i32(static_cast<const int32_t *>(v->col[t.table_id][c]) + t.first_row,
+                                  t.row_count - t.first_row,
+                                  stats_dev + (t.table_id * kStatCols + c) * 2, e->num_sms, e->copy);
     }
     CK(cudaEventRecord(pend.t1, e->copy));
     // ---- in-place updates: upload every update's row ids and values first (one arena region;
@@ -652,7 +653,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
             const auto *rows_d = reinterpret_cast<const uint32_t *>(upd_dev + upd_off[i]);
             const void *vals_d = upd_dev + upd_off[i] + round_up16(u.n * 4);
             launch_apply_updates(cs.alt->ptr, (uint32_t)es, next_bits, rows_d, vals_d, u.n, e->num_sms, e->copy);
-            if (u.table_id != H2TAP_T_ITEM && u.column_id < (uint32_t)kStatCols)  // zone map: widen
+            if (u.column_id < (uint32_t)stat_cols(u.table_id))  // zone map: widen
                 launch_minmax_i32(static_cast<const int32_t *>(vals_d), u.n,
                                   stats_dev + (u.table_id * kStatCols + u.column_id) * 2, e->num_sms, e->copy);
         }
@@ -752,6 +753,10 @@ struct QueryCtx {
     unsigned int *tie_dev = nullptr;
     bool q18_sorted_on_host_sync = false;   // world > 1 path already knows nout
     uint64_t nout_host = 0;
+    // NEXT-2: Q14 / Q12 / Q4
+    Q14Scratch q14{};
+    SmallGroups sg{};
+    unsigned int *err = nullptr;
 };
 
 void *dev_block(h2tap_engine *e, QueryCtx &q, size_t bytes) {
@@ -1146,11 +1151,228 @@ void finish_q18(h2tap_engine *e, QueryCtx &q) {
     release_dev_blocks(e, q);
 }
 
+// ---- NEXT-2: CH Q14 (order_line ⋈ item), Q12 (orders ⋈ order_line), Q4 (orders ⋉ order_line)
+struct SgSmall { unsigned long long ngroups; unsigned int flags, err; };
+struct Q14Small { long long out[3]; double promo; unsigned int err; };
+
+void raise_join_err(unsigned int err, const char *plan) {
+    if (err & kErrDupOrders) raise(H2TAP_EDUPKEY, "%s: duplicate orders primary key (w, d, o_id)", plan);
+    if (err & kErrDupItem) raise(H2TAP_EDUPKEY, "%s: duplicate item primary key i_id", plan);
+    if (err & kErrDomain) raise(H2TAP_EPLAN, "%s: join key outside the supported domain", plan);
+}
+
+void launch_q14_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
+    const int OL = H2TAP_T_ORDER_LINE, I = H2TAP_T_ITEM;
+    need_cols(v, OL, {H2TAP_OL_DELIVERY_D, H2TAP_OL_I_ID, H2TAP_OL_AMOUNT}, "Q14");
+    need_cols(v, I, {H2TAP_I_ID, H2TAP_I_DATA_P2}, "Q14");
+    const uint64_t n_i = v.n[I];
+    ItemMap m{};
+    if (n_i) {  // i_id box from the item zone map (R31)
+        if (!v.has_stats[I]) raise(H2TAP_EPLAN, "Q14: no statistics for item");
+        m.i0 = v.smin[I][0];
+        m.range = (unsigned long long)((long long)v.smax[I][0] - v.smin[I][0] + 1);
+        if (m.range > (1ull << 28)) raise(H2TAP_EPLAN, "Q14: item ids span %llu values (> 2^28)", m.range);
+        m.words = (m.range + 15) / 16;
+    }
+    m.bits = static_cast<unsigned int *>(e->arena.get("q14.map", 4 * (m.words + 1)));
+    Q14Scratch &s = q.q14;
+    s.block_part = static_cast<long long *>(e->arena.get("q14.part", 24ull * q14_max_blocks(e->num_sms)));
+    s.done_counter = static_cast<unsigned int *>(e->arena.get("q14.counter", 64, true, e->compute));
+    s.out = static_cast<long long *>(e->arena.get("q14.out", 32));
+    s.promo = static_cast<double *>(dev_block(e, q, 8));
+    q.err = static_cast<unsigned int *>(e->arena.get("q14.err", 64));
+    CK(cudaMemsetAsync(q.err, 0, 4, e->compute));
+    q.r->plan_flags = m.words <= 16384 ? 4u : 0u;  // bit2: item map held in shared memory
+    e->prof.run("q14_item_map", [&] {
+        launch_item_map(colp<int32_t>(v, I, H2TAP_I_ID), colp<int32_t>(v, I, H2TAP_I_DATA_P2), n_i,
+                        (int32_t)q.p[2], m, q.err, e->num_sms, e->compute);
+    });
+    e->prof.run("q14_scan_join_sum", [&] {
+        launch_q14(colp<int64_t>(v, OL, H2TAP_OL_DELIVERY_D), colp<int32_t>(v, OL, H2TAP_OL_I_ID),
+                   colp<int64_t>(v, OL, H2TAP_OL_AMOUNT), v.n[OL], q.p[0], q.p[1], m, s, e->num_sms,
+                   e->compute);
+        CK(cudaGetLastError());
+    });
+    if (e->world > 1)
+        e->prof.run("q14_allreduce", [&] {
+            NK(ncclAllReduce(s.out, s.out, 3, ncclInt64, ncclSum, e->comm, e->compute));
+        });
+    e->prof.run("q14_finalize", [&] { launch_q14_finalize(s, e->compute); });
+    auto *sm = static_cast<Q14Small *>(q.small.first);
+    CK(cudaMemcpyAsync(sm->out, s.out, 24, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaMemcpyAsync(&sm->promo, s.promo, 8, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaMemcpyAsync(&sm->err, q.err, 4, cudaMemcpyDeviceToHost, e->compute));
+}
+
+void finish_q14(h2tap_engine *e, QueryCtx &q) {
+    ResultImpl *r = q.r.get();
+    const auto *sm = static_cast<const Q14Small *>(q.small.first);
+    raise_join_err(sm->err, "Q14");
+    r->nrows = 1;
+    const bool null = sm->out[2] == 0;  // SUM over no joined row IS NULL -> NULL ratio (R30)
+    auto *blk = static_cast<long long *>(result_block(r, 32));
+    if (r->on_device) {
+        CK(cudaMemcpy(blk, sm->out, 24, cudaMemcpyHostToDevice));
+        add_col(r, "promo_revenue", H2TAP_F64, q.q14.promo);
+        give_blocks_to_result(q);
+    } else {
+        std::memcpy(blk, sm->out, 24);
+        std::memcpy(blk + 3, &sm->promo, 8);
+        add_col(r, "promo_revenue", H2TAP_F64, blk + 3);
+        release_dev_blocks(e, q);
+    }
+    r->null_store.back().assign(1, null ? 1 : 0);
+    add_col(r, "sum_promo", H2TAP_I64, blk);
+    r->null_store.back().assign(1, null ? 1 : 0);
+    add_col(r, "sum_amount", H2TAP_I64, blk + 1);
+    r->null_store.back().assign(1, null ? 1 : 0);
+    add_col(r, "count_rows", H2TAP_I64, blk + 2);
+}
+
+// small-group tables (dense | gtag | gacc contiguous, so one allgather moves them) + outputs
+void sg_setup(h2tap_engine *e, QueryCtx &q) {
+    SmallGroups &g = q.sg;
+    const bool fresh = !e->arena.bufs.count("sg.tables");
+    auto *t = static_cast<unsigned long long *>(e->arena.get("sg.tables", 8ull * (3 * kSgDense + 4 * kSgSlots)));
+    g.dense = t;
+    g.gtag = t + 3 * kSgDense;
+    g.gacc = g.gtag + kSgSlots;
+    g.flags = static_cast<unsigned int *>(e->arena.get("sg.flags", 64));
+    g.ngroups = static_cast<unsigned long long *>(e->arena.get("sg.ngroups", 64));
+    const size_t maxg = kSgSlots + kSgDense;
+    g.o_key = static_cast<int32_t *>(dev_block(e, q, 4 * maxg));
+    g.o_a = static_cast<long long *>(dev_block(e, q, 8 * maxg));
+    g.o_b = static_cast<long long *>(dev_block(e, q, 8 * maxg));
+    if (fresh) launch_sg_reset(g, e->compute);  // the emit kernel re-clears after every query
+    q.err = static_cast<unsigned int *>(e->arena.get("sg.err", 64));
+    CK(cudaMemsetAsync(q.err, 0, 4, e->compute));
+}
+
+void sg_merge_and_emit(h2tap_engine *e, QueryCtx &q, const char *name) {
+    SmallGroups &g = q.sg;
+    if (e->world > 1) {  // a7: every rank's tables to every rank, folded into the local one
+        const size_t words = 3 * kSgDense + 4 * kSgSlots;
+        auto *all = static_cast<unsigned long long *>(e->arena.get("sg.all", 8ull * words * e->world));
+        e->prof.run((std::string(name) + "_allgather").c_str(), [&] {
+            NK(ncclAllGather(g.dense, all, words, ncclUint64, e->comm, e->compute));
+        });
+        for (int k = 0; k < e->world; ++k)
+            if (k != e->rank) {
+                const unsigned long long *t = all + (size_t)k * words;
+                launch_sg_merge(t, t + 3 * kSgDense, t + 3 * kSgDense + kSgSlots, g, e->compute);
+            }
+    }
+    e->prof.run((std::string(name) + "_emit").c_str(), [&] { launch_sg_emit(g, e->compute); });
+    auto *sm = static_cast<SgSmall *>(q.small.first);
+    CK(cudaMemcpyAsync(&sm->ngroups, g.ngroups, 8, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaMemcpyAsync(&sm->flags, g.flags, 4, cudaMemcpyDeviceToHost, e->compute));
+    CK(cudaMemcpyAsync(&sm->err, q.err, 4, cudaMemcpyDeviceToHost, e->compute));
+}
+
+JoinIndex plan_orders_index(h2tap_engine *e, const View &v, QueryCtx &q, const char *plan) {
+    const int O = H2TAP_T_ORDERS;
+    JoinIndex jo = plan_index(e, v, O, q.flags & H2TAP_QUERY_HASH_JOIN, "ch.jo");
+    q.r->plan_flags = jo.dense ? 1u : 0u;
+    (void)plan;
+    return jo;
+}
+
+void launch_q12_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
+    const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS;
+    need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_DELIVERY_D}, "Q12");
+    need_cols(v, O, {H2TAP_O_W_ID, H2TAP_O_D_ID, H2TAP_O_ID, H2TAP_O_OL_CNT, H2TAP_O_CARRIER_ID, H2TAP_O_ENTRY_D}, "Q12");
+    sg_setup(e, q);
+    const JoinIndex jo = plan_orders_index(e, v, q, "Q12");
+    e->prof.run("q12_build", [&] {
+        launch_jx_build_orders(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
+                               colp<int32_t>(v, O, H2TAP_O_ID), v.n[O], jo, q.err, nullptr, e->num_sms, e->compute);
+    });
+    e->prof.run("q12_probe_groupby", [&] {
+        if (v.n[OL])
+            launch_q12_probe(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
+                             colp<int32_t>(v, OL, H2TAP_OL_O_ID), colp<int64_t>(v, OL, H2TAP_OL_DELIVERY_D),
+                             v.n[OL], jo, colp<int64_t>(v, O, H2TAP_O_ENTRY_D), colp<int32_t>(v, O, H2TAP_O_CARRIER_ID),
+                             colp<int32_t>(v, O, H2TAP_O_OL_CNT), q.p[0], q.sg, e->num_sms, e->compute);
+        CK(cudaGetLastError());
+    });
+    sg_merge_and_emit(e, q, "q12");
+}
+
+void launch_q4_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
+    const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS;
+    need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_DELIVERY_D}, "Q4");
+    need_cols(v, O, {H2TAP_O_W_ID, H2TAP_O_D_ID, H2TAP_O_ID, H2TAP_O_OL_CNT, H2TAP_O_ENTRY_D}, "Q4");
+    sg_setup(e, q);
+    const JoinIndex jo = plan_orders_index(e, v, q, "Q4");
+    auto *mark = static_cast<uint8_t *>(e->arena.get("q4.mark", std::max<uint64_t>(v.n[O], 1) + 16));
+    e->prof.run("q4_build", [&] {
+        launch_jx_build_orders(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
+                               colp<int32_t>(v, O, H2TAP_O_ID), v.n[O], jo, q.err, mark, e->num_sms, e->compute);
+    });
+    struct Marks : PhaseMarks {
+        Prof &p;
+        cudaEvent_t a = nullptr;
+        std::string name;
+        explicit Marks(Prof &pr) : p(pr) {}
+        void begin(const char *nm) override {
+            if (!p.on) return;
+            name = nm;
+            a = p.ev();
+            CK(cudaEventRecord(a, p.st));
+        }
+        void end() override {
+            if (!p.on) return;
+            cudaEvent_t b = p.ev();
+            CK(cudaEventRecord(b, p.st));
+            p.marks.push_back({name, {a, b}});
+        }
+    } marks(e->prof);
+    launch_q4(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
+              colp<int32_t>(v, OL, H2TAP_OL_O_ID), colp<int64_t>(v, OL, H2TAP_OL_DELIVERY_D), v.n[OL], jo,
+              colp<int64_t>(v, O, H2TAP_O_ENTRY_D), colp<int32_t>(v, O, H2TAP_O_OL_CNT), v.n[O], q.p[0], q.p[1],
+              mark, q.sg, e->num_sms, e->compute, &marks);
+    CK(cudaGetLastError());
+    sg_merge_and_emit(e, q, "q4");
+}
+
+void finish_groups(h2tap_engine *e, QueryCtx &q, const char *plan, const char *a_name, const char *b_name) {
+    ResultImpl *r = q.r.get();
+    const auto *sm = static_cast<const SgSmall *>(q.small.first);
+    raise_join_err(sm->err, plan);
+    if (sm->flags & 1) {
+        CK(cudaMemsetAsync(q.sg.flags, 0, 4, e->compute));
+        raise(H2TAP_ENOMEM, "%s: more than %d distinct o_ol_cnt groups", plan, kSgSlots + kSgDense);
+    }
+    const uint64_t ng = sm->ngroups;
+    r->nrows = ng;
+    struct { const char *name; uint32_t type; const void *src; size_t es; } cols[] = {
+        {"o_ol_cnt", H2TAP_I32, q.sg.o_key, 4}, {a_name, H2TAP_I64, q.sg.o_a, 8}, {b_name, H2TAP_I64, q.sg.o_b, 8}};
+    const int ncols = b_name ? 3 : 2;
+    if (r->on_device) {
+        for (int i = 0; i < ncols; ++i) add_col(r, cols[i].name, cols[i].type, cols[i].src);
+        give_blocks_to_result(q);
+        return;
+    }
+    for (int i = 0; i < ncols; ++i) {
+        void *dst = result_block(r, ng * cols[i].es);
+        if (ng) CK(cudaMemcpyAsync(dst, cols[i].src, ng * cols[i].es, cudaMemcpyDeviceToHost, e->compute));
+        add_col(r, cols[i].name, cols[i].type, dst);
+    }
+    sync_compute(e);
+    release_dev_blocks(e, q);
+}
+
 // CH-benCHmark constants as int64 µs UTC / cents (R4, R6).
 constexpr int64_t kQ1Cutoff = 1167696000000000LL;   // 2007-01-02 00:00:00
 constexpr int64_t kQ6DLo = 915148800000000LL;       // 1999-01-01 00:00:00
 constexpr int64_t kQ6DHi = 1577836800000000LL;      // 2020-01-01 00:00:00
 constexpr int64_t kQ18Having = 20000;               // 200.00
+constexpr int64_t kQ14DLo = 1167696000000000LL;     // 2007-01-02 00:00:00
+constexpr int64_t kQ14DHi = 1577923200000000LL;     // 2020-01-02 00:00:00
+constexpr int64_t kQ14Prefix = 0x5052;              // 'P' << 8 | 'R'  (LIKE 'PR%')
+constexpr int64_t kQ12DHi = 1577836800000000LL;     // 2020-01-01 00:00:00
+constexpr int64_t kQ4ELo = 1167696000000000LL;      // 2007-01-02 00:00:00
+constexpr int64_t kQ4EHi = 1325462400000000LL;      // 2012-01-02 00:00:00
 
 h2tap_status parse_query(const h2tap_query &in, QueryCtx &q) {
     uint32_t want;
@@ -1158,6 +1380,9 @@ h2tap_status parse_query(const h2tap_query &in, QueryCtx &q) {
         case H2TAP_Q1: want = 1; q.p[0] = kQ1Cutoff; break;
         case H2TAP_Q6: want = 4; q.p[0] = kQ6DLo; q.p[1] = kQ6DHi; q.p[2] = 1; q.p[3] = 100000; break;
         case H2TAP_Q18: want = 1; q.p[0] = kQ18Having; break;
+        case H2TAP_Q14: want = 3; q.p[0] = kQ14DLo; q.p[1] = kQ14DHi; q.p[2] = kQ14Prefix; break;
+        case H2TAP_Q12: want = 1; q.p[0] = kQ12DHi; break;
+        case H2TAP_Q4: want = 2; q.p[0] = kQ4ELo; q.p[1] = kQ4EHi; break;
         default: return fail(H2TAP_EINVAL, "unknown plan id %u", in.plan_id);
     }
     if (in.nparams) {
@@ -1218,6 +1443,9 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
                 case H2TAP_Q1: finish_q1(e, q); break;
                 case H2TAP_Q6: finish_q6(e, q); break;
                 case H2TAP_Q18: finish_q18(e, q); break;
+                case H2TAP_Q14: finish_q14(e, q); break;
+                case H2TAP_Q12: finish_groups(e, q, "Q12", "high_line_count", "low_line_count"); break;
+                case H2TAP_Q4: finish_groups(e, q, "Q4", "order_count", nullptr); break;
             }
         }
     };
@@ -1238,6 +1466,9 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
             case H2TAP_Q1: launch_q1_plan(e, *v, q); break;
             case H2TAP_Q6: launch_q6_plan(e, *v, q); break;
             case H2TAP_Q18: launch_q18_plan(e, *v, q); break;
+            case H2TAP_Q14: launch_q14_plan(e, *v, q); break;
+            case H2TAP_Q12: launch_q12_plan(e, *v, q); break;
+            case H2TAP_Q4: launch_q4_plan(e, *v, q); break;
         }
         CK(cudaEventRecord(q.end, e->compute));
         q.launches = launches_total() - q.launches0;

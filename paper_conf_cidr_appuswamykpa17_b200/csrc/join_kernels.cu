@@ -16,69 +16,14 @@
 
 #include "bulk_pipeline.cuh"
 #include "cache_hints.cuh"
+#include "join_index.cuh"
 #include "kernels.cuh"
 
 namespace h2tap {
 namespace {
+using namespace jx;
 
 constexpr unsigned kFull = 0xffffffffu;
-
-__device__ __forceinline__ unsigned long long fmix64(unsigned long long k) {
-    k ^= k >> 33; k *= 0xff51afd7ed558ccdull; k ^= k >> 33; k *= 0xc4ceb9fe1a85ec53ull; k ^= k >> 33;
-    return k;
-}
-
-// (w, d, id) -> 64-bit key, injective on the supported domain (R16).
-__device__ __forceinline__ bool pack_key(int w, int d, int id, unsigned long long &k) {
-    k = ((unsigned long long)(unsigned)w << 40) | ((unsigned long long)(unsigned)d << 32) |
-        (unsigned long long)(unsigned)id;
-    return ((unsigned)w < (1u << 23)) & ((unsigned)d < 256u) & (id >= 0);
-}
-
-// Dense slot of (w, d, id) in the index's box, or false when outside it.
-__device__ __forceinline__ bool dense_slot(const JoinIndex &j, int w, int d, int id,
-                                          unsigned long long &slot) {
-    const unsigned dw = (unsigned)(w - j.w0), dd = (unsigned)(d - j.d0), dk = (unsigned)(id - j.k0);
-    slot = ((unsigned long long)dw * j.nd + dd) * j.nk + dk;
-    return (dw < j.nw) & (dd < j.nd) & (dk < j.nk);
-}
-
-// Insert; returns false on a key outside the supported domain. Duplicates set `dupbit`.
-__device__ __forceinline__ bool jx_insert(const JoinIndex &j, int w, int d, int id, unsigned int row,
-                                          unsigned int *err, unsigned int dupbit) {
-    if (j.dense) {
-        unsigned long long s;
-        if (!dense_slot(j, w, d, id, s)) return false;  // stats must cover every build row
-        if (atomicCAS(j.slots + s, kNoRow, row) != kNoRow) atomicOr(err, dupbit);
-        return true;
-    }
-    unsigned long long key;
-    if (!pack_key(w, d, id, key)) return false;
-    unsigned long long h = fmix64(key) & j.mask;
-    while (true) {
-        const unsigned long long prev = atomicCAS(&j.ht[h].key, kEmpty, key);
-        if (prev == kEmpty) { j.ht[h].row = row; return true; }
-        if (prev == key) { atomicOr(err, dupbit); return true; }
-        h = (h + 1) & j.mask;
-    }
-}
-
-__device__ __forceinline__ unsigned int jx_lookup(const JoinIndex &j, int w, int d, int id) {
-    if (j.dense) {
-        unsigned long long s;
-        if (!dense_slot(j, w, d, id, s)) return kNoRow;  // outside the build box: no match
-        return __ldcg(j.slots + s);
-    }
-    unsigned long long key;
-    if (!pack_key(w, d, id, key)) return kNoRow;  // no build key can lie outside the domain
-    unsigned long long h = fmix64(key) & j.mask;
-    while (true) {
-        const ulonglong2 s = __ldcg(reinterpret_cast<const ulonglong2 *>(j.ht + h));
-        if (s.x == key) return (unsigned int)s.y;
-        if (s.x == kEmpty) return kNoRow;
-        h = (h + 1) & j.mask;
-    }
-}
 
 unsigned grid_for(uint64_t work, int threads, int num_sms, int per_sm) {
     uint64_t want = (work + threads - 1) / threads;
@@ -89,14 +34,7 @@ unsigned grid_for(uint64_t work, int threads, int num_sms, int per_sm) {
 
 // ------------------------------------------------------------------- init --
 // Empties both join indexes, zeroes the group accumulators and the counters: one launch.
-__host__ __device__ __forceinline__ uint64_t jx_words(const JoinIndex &j) {  // 16-byte units
-    return j.dense ? (j.range + 3) / 4 : j.mask + 1;
-}
-__device__ __forceinline__ void jx_clear(const JoinIndex &j, uint64_t i) {
-    if (j.dense) reinterpret_cast<uint4 *>(j.slots)[i] = make_uint4(kNoRow, kNoRow, kNoRow, kNoRow);
-    else reinterpret_cast<ulonglong2 *>(j.ht)[i] = make_ulonglong2(kEmpty, 0ull);
-}
-
+// Empties both join indexes, zeroes the group accumulators and the counters: one launch.
 __global__ void q18_init_kernel(Q18Scratch s) {
     const uint64_t a = jx_words(s.jo), b = jx_words(s.jc);
     const uint64_t total = a + b;  // (the accumulators are zeroed by the build, row by row)

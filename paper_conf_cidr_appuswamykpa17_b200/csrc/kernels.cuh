@@ -60,7 +60,7 @@ struct HtSlot { unsigned long long key; unsigned int row; unsigned int pad; };  
 constexpr unsigned long long kEmpty = ~0ull;
 constexpr unsigned int kNoRow = 0xffffffffu;
 struct Q18Acc { long long sum; unsigned int cnt; unsigned int pad; };          // 16 B
-enum : unsigned int { kErrDupOrders = 1u, kErrDupCustomer = 2u, kErrDomain = 4u };
+enum : unsigned int { kErrDupOrders = 1u, kErrDupCustomer = 2u, kErrDomain = 4u, kErrDupItem = 8u };
 
 // Join index on a (w, d, id) primary key -> row. Two layouts, chosen per query by the planner
 // from the snapshot's column statistics:
@@ -207,6 +207,48 @@ void launch_apply_updates(void *col, uint32_t es, uint32_t *bits, const uint32_t
 // ---------------------------------------------------------------- helpers --
 // Every launcher counts the kernels it launches (reported per query as kernel_launches).
 void count_launches(int n);
+
+// ------------------------------------------- NEXT-2: CH Q14 / Q12 / Q4 (ch_kernels.cu) --
+// GROUP BY o_ol_cnt with counters (a, b, rows) per group: keys in [0, kSgDense) in thread-private
+// shared memory, others in a global open-addressing table of kSgSlots groups.
+constexpr int kSgDense = 16;
+constexpr int kSgSlots = 2048;
+struct SmallGroups {
+    unsigned long long *dense;     // [3 * kSgDense]: a, b, rows of key k at 3k..3k+2
+    unsigned long long *gtag;      // [kSgSlots]: 0 = empty, else (1 << 32 | (u32)key)
+    unsigned long long *gacc;      // [3 * kSgSlots]
+    unsigned int *flags;           // [1]: bit0 = table full
+    int32_t *o_key; long long *o_a, *o_b; unsigned long long *ngroups;  // output ranked by key
+};
+void launch_sg_reset(const SmallGroups &g, cudaStream_t st);  // once, at allocation
+void launch_sg_emit(const SmallGroups &g, cudaStream_t st);   // rank + write; re-clears the tables
+void launch_sg_merge(const unsigned long long *dense, const unsigned long long *gtag,
+                     const unsigned long long *gacc, const SmallGroups &g, cudaStream_t st);
+// orders (w, d, o_id) join index alone: clear + insert (and zero mark[] for Q4 when non-null)
+void launch_jx_build_orders(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
+                            const JoinIndex &jo, unsigned int *err, uint8_t *mark, int num_sms,
+                            cudaStream_t st);
+void launch_q12_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o, const int64_t *ol_dl,
+                      uint64_t n_ol, const JoinIndex &jo, const int64_t *o_entry, const int32_t *o_carrier,
+                      const int32_t *o_cnt, int64_t d_hi, const SmallGroups &g, int num_sms, cudaStream_t st);
+void launch_q4(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o, const int64_t *ol_dl,
+               uint64_t n_ol, const JoinIndex &jo, const int64_t *o_entry, const int32_t *o_cnt,
+               uint64_t n_o, int64_t e_lo, int64_t e_hi, uint8_t *mark, const SmallGroups &g,
+               int num_sms, cudaStream_t st, PhaseMarks *marks);
+// Q14: item map, 2 bits per i_id in [i0, i0 + range): bit0 exists, bit1 i_data prefix matches
+struct ItemMap { unsigned int *bits; long long i0; unsigned long long range, words; };
+void launch_item_map(const int32_t *i_id, const int32_t *p2, uint64_t n, int32_t prefix2, const ItemMap &m,
+                     unsigned int *err, int num_sms, cudaStream_t st);
+struct Q14Scratch {
+    long long *block_part;         // [3 * q14_max_blocks]
+    unsigned int *done_counter;    // [1], zero-initialised once, self-resetting
+    long long *out;                // [3]: sum_promo, sum_amount, count
+    double *promo;                 // [1]
+};
+int q14_max_blocks(int num_sms);
+void launch_q14(const int64_t *deliv, const int32_t *i_id, const int64_t *amt, uint64_t n, int64_t d_lo,
+                int64_t d_hi, const ItemMap &m, const Q14Scratch &s, int num_sms, cudaStream_t st);
+void launch_q14_finalize(const Q14Scratch &s, cudaStream_t st);
 uint64_t launches_total();
 
 }  // namespace h2tap

@@ -29,8 +29,8 @@ def h():
 def _hot_updates(h, upd):
     """Keep the updates of columns the hot path loads (o_carrier_id is not one of them)."""
     hot = {}
-    for spec in h.plan_columns().values():
-        for t, cols in spec.items():
+    for plan in h.HOT_PATH_PLANS:
+        for t, cols in h.plan_columns()[plan].items():
             hot.setdefault(t, set()).update(cols)
     return {t: {c: v for c, v in cols.items() if c in hot.get(t, ())} for t, cols in upd.items()}
 
