@@ -6,11 +6,12 @@
 //       (25 KB for TPC-C's 100 000 items); int64 sums, last-block fold, promo ratio in double.
 //  Q12  orders ⋈ order_line GROUP BY o_ol_cnt: stream (w, d, o, delivery) per line, one lookup of
 //       the orders join index per run of equal keys inside a lane, gather (entry, carrier,
-//       ol_cnt), count per group in thread-private shared-memory counters.
+//       ol_cnt), count per group in thread-private 16-bit shared-memory counters.
 //  Q4   orders ⋉ order_line (EXISTS): the same stream marks orders rows that have a qualifying
 //       line (idempotent byte store), then one pass over orders counts marked rows per o_ol_cnt.
 // The paper gives no plans for these queries (it evaluates TPC-H Q6 only);
 // like the hot path they run on an epoch's snapshot (L555-572). DESIGN.md §4.8.
+#include <algorithm>
 #include <cstdint>
 #include <cuda_runtime.h>
 
@@ -38,11 +39,13 @@ unsigned grid_for(uint64_t work, int threads, int num_sms, int per_sm) {
 }
 
 // ============================================================ small groups ==
-// GROUP BY o_ol_cnt with three counters per group (a, b, rows). Keys in [0, kSgDense) are counted
-// in thread-private shared memory (no atomics) and folded once per block; other keys go to a
-// global open-addressing table (atomics; TPC-C never produces them).
+// GROUP BY o_ol_cnt with three counters per group (a, b, rows). Per warp step the lanes with a
+// contribution are grouped by key (__match_any_sync); one leader per distinct key adds the
+// group's popcounts to the block's shared counters (keys in [0, kSgDense)) or to a global
+// open-addressing table (other keys; TPC-C never produces them). The block's counters are folded
+// into g.dense once at the end. Shared memory stays tiny, so occupancy is not limited by it.
 struct SgSmem {
-    unsigned int c[3][kSgDense][kThreads];  // [counter][key][thread]: lane-distinct banks
+    unsigned int c[kSgDense][3];
 };
 
 __device__ __forceinline__ unsigned int hash32(unsigned int x) {
@@ -68,31 +71,65 @@ __device__ void sg_global_add(const SmallGroups &g, int key, unsigned long long 
 }
 
 __device__ __forceinline__ void sg_clear(SgSmem &S) {
-    unsigned int *p = &S.c[0][0][0];
-    for (int i = threadIdx.x; i < 3 * kSgDense * kThreads; i += blockDim.x) p[i] = 0;
+    for (int i = threadIdx.x; i < 3 * kSgDense; i += blockDim.x) (&S.c[0][0])[i] = 0;
 }
 
-__device__ __forceinline__ void sg_add(SgSmem &S, const SmallGroups &g, int key, unsigned a, unsigned b) {
+// Warp-collective: every lane calls it (ok = this lane contributes a row to group `key`, with
+// flags a and b). One shared (or global) update per distinct key of the warp.
+__device__ __forceinline__ void sg_warp_add(SgSmem &S, const SmallGroups &g, bool ok, int key, bool a, bool b) {
+    const unsigned okm = __ballot_sync(kFull, ok);
+    if (!okm) return;
+    const unsigned am = __ballot_sync(kFull, ok && a), bm = __ballot_sync(kFull, ok && b);
+    if (!ok) return;
+    const unsigned grp = __match_any_sync(okm, key);
+    if ((int)(threadIdx.x & 31) != __ffs(grp) - 1) return;
+    const unsigned na = __popc(grp & am), nb = __popc(grp & bm), nr = __popc(grp);
     if ((unsigned)key < (unsigned)kSgDense) {
-        S.c[0][key][threadIdx.x] += a;
-        S.c[1][key][threadIdx.x] += b;
-        S.c[2][key][threadIdx.x] += 1;
+        if (na) atomicAdd(&S.c[key][0], na);
+        if (nb) atomicAdd(&S.c[key][1], nb);
+        atomicAdd(&S.c[key][2], nr);
+    } else {
+        sg_global_add(g, key, na, nb, nr);
+    }
+}
+
+// Thread-private variant for the probe (Q12): c[counter][key][thread] in 16-bit counters (a thread
+// sees at most 2^31 / (148 * 8 * 256) < 65 536 rows), lane-distinct halves of a word, no atomics.
+struct SgPriv {
+    unsigned short c[3][kSgDense][kThreads];
+};
+__device__ __forceinline__ void sgp_clear(SgPriv &P) {
+    unsigned int *p = reinterpret_cast<unsigned int *>(&P.c[0][0][0]);
+    for (int i = threadIdx.x; i < 3 * kSgDense * kThreads / 2; i += blockDim.x) p[i] = 0;
+}
+__device__ __forceinline__ void sgp_add(SgPriv &P, const SmallGroups &g, int key, bool a, bool b) {
+    if ((unsigned)key < (unsigned)kSgDense) {
+        P.c[0][key][threadIdx.x] += a;
+        P.c[1][key][threadIdx.x] += b;
+        P.c[2][key][threadIdx.x] += 1;
     } else {
         sg_global_add(g, key, a, b, 1);
     }
 }
-
-// fold the block's private counters into g.dense: warp w sums rows w, w+8, ... (lanes stride the
-// 256 threads), one 64-bit atomic per non-zero (counter, key)
-__device__ void sg_flush(SgSmem &S, const SmallGroups &g) {
+// warp r sums counter row r (over the 256 threads), one 64-bit atomic per non-zero row
+__device__ void sgp_flush(SgPriv &P, const SmallGroups &g) {
     __syncthreads();
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     for (int r = warp; r < 3 * kSgDense; r += blockDim.x / 32) {
-        const unsigned int *row = &S.c[r / kSgDense][r % kSgDense][0];
+        const unsigned short *row = &P.c[r / kSgDense][r % kSgDense][0];
         long long v = 0;
         for (int t = lane; t < kThreads; t += 32) v += row[t];
         v = warp_sum64(v);
         if (lane == 0 && v) atomicAdd(g.dense + (r % kSgDense) * 3 + r / kSgDense, (unsigned long long)v);
+    }
+}
+
+// fold the block's counters into g.dense: one 64-bit atomic per non-zero (key, counter)
+__device__ void sg_flush(SgSmem &S, const SmallGroups &g) {
+    __syncthreads();
+    for (int i = threadIdx.x; i < 3 * kSgDense; i += blockDim.x) {
+        const unsigned v = (&S.c[0][0])[i];
+        if (v) atomicAdd(g.dense + i, (unsigned long long)v);
     }
 }
 
@@ -183,18 +220,23 @@ __global__ void jx_build_orders_kernel(const int32_t *__restrict__ o_w, const in
 }
 
 // ======================================================= Q12 / Q4 probes ==
-// Each lane owns 4 consecutive order_line rows (128-bit loads of w, d, o, two of delivery); the
-// orders row is looked up once per run of equal keys inside the lane (lines of an order are
-// adjacent), and the row's (entry, carrier, ol_cnt) gathered once per lookup.
+// Each lane owns 4 consecutive order_line rows (128-bit loads of w, d, o, two of delivery). The
+// lane first issues the orders-index lookups of every run start among its 4 rows (independent
+// loads, all in flight together; lines of an order are adjacent so ~1.4 per lane), then the
+// gathers of the looked-up rows' fields, then evaluates — two memory round trips per 4 rows
+// instead of one chain per row.
 struct OrderCols { const int64_t *entry; const int32_t *carrier, *cnt; };
 
-template <class RowFn>
-__device__ __forceinline__ void probe_rows(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ ol_d,
-                                           const int32_t *__restrict__ ol_o, const int64_t *__restrict__ ol_dl,
-                                           uint64_t n, const JoinIndex &jo, RowFn &&fn) {
+// fn(row[4], dl[4], valid): called once per lane per 4 rows (warp-uniform; rows past the end
+// have valid = false). row[j] = orders row of line j or kNoRow.
+template <class Fn>
+__device__ __forceinline__ void probe_rows4(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ ol_d,
+                                            const int32_t *__restrict__ ol_o, const int64_t *__restrict__ ol_dl,
+                                            uint64_t n, const JoinIndex &jo, Fn &&fn) {
     const uint64_t nvec = n >> 2;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    const unsigned lane = threadIdx.x & 31;
+    uint64_t base = (uint64_t)blockIdx.x * blockDim.x + (threadIdx.x & ~31u);
     int4 nW = make_int4(0, 0, 0, 0), nD = nW, nO = nW;
     longlong2 nL0 = make_longlong2(0, 0), nL1 = nL0;
     auto load = [&](uint64_t x) {
@@ -206,53 +248,70 @@ __device__ __forceinline__ void probe_rows(const int32_t *__restrict__ ol_w, con
             nL1 = __ldcs(reinterpret_cast<const longlong2 *>(ol_dl) + 2 * x + 1);
         }
     };
-    load(v);
-    for (; v < nvec; v += stride) {
-        const int w[4] = {nW.x, nW.y, nW.z, nW.w}, d[4] = {nD.x, nD.y, nD.z, nD.w},
-                  o[4] = {nO.x, nO.y, nO.z, nO.w};
+    load(base + lane);
+    for (; base < nvec; base += stride) {
+        const bool valid = base + lane < nvec;
+        const int4 W = nW, D = nD, O = nO;
         const long long dl[4] = {nL0.x, nL0.y, nL1.x, nL1.y};
-        load(v + stride);  // next group's loads in flight while this one is probed
-        unsigned int row = kNoRow;
-#pragma unroll
-        for (int j = 0; j < 4; ++j) {
-            if (j == 0 || w[j] != w[j - 1] || d[j] != d[j - 1] || o[j] != o[j - 1])
-                row = jx_lookup(jo, w[j], d[j], o[j]);
-            fn(row, dl[j]);
-        }
+        load(base + stride + lane);  // next group's loads in flight while this one is probed
+        const bool s1 = (W.y != W.x) | (D.y != D.x) | (O.y != O.x);
+        const bool s2 = (W.z != W.y) | (D.z != D.y) | (O.z != O.y);
+        const bool s3 = (W.w != W.z) | (D.w != D.z) | (O.w != O.z);
+        unsigned int r[4];
+        r[0] = valid ? jx_lookup(jo, W.x, D.x, O.x) : kNoRow;
+        r[1] = valid && s1 ? jx_lookup(jo, W.y, D.y, O.y) : kNoRow;
+        r[2] = valid && s2 ? jx_lookup(jo, W.z, D.z, O.z) : kNoRow;
+        r[3] = valid && s3 ? jx_lookup(jo, W.w, D.w, O.w) : kNoRow;
+        if (!s1) r[1] = r[0];
+        if (!s2) r[2] = r[1];
+        if (!s3) r[3] = r[2];
+        fn(r, dl, valid);
     }
-    // ragged tail (< 4 rows): the first threads, one row each
-    const uint64_t t = 4 * nvec + (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
-    if (t < n) fn(jx_lookup(jo, ol_w[t], ol_d[t], ol_o[t]), ol_dl[t]);
+    // ragged tail (< 4 rows): the first warp of block 0, one row per lane (warp-uniform call)
+    if (blockIdx.x == 0 && threadIdx.x < 32) {
+        const uint64_t t = 4 * nvec + lane;
+        const bool valid = t < n;
+        unsigned int r[4] = {valid ? jx_lookup(jo, ol_w[t], ol_d[t], ol_o[t]) : kNoRow, kNoRow, kNoRow, kNoRow};
+        const long long dl[4] = {valid ? ol_dl[t] : 0ll, kNullTs, kNullTs, kNullTs};
+        fn(r, dl, valid);
+    }
 }
 
 __global__ void __launch_bounds__(kThreads)
 q12_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ ol_d,
                  const int32_t *__restrict__ ol_o, const int64_t *__restrict__ ol_dl, uint64_t n,
                  JoinIndex jo, OrderCols oc, long long d_hi, SmallGroups g) {
-    extern __shared__ __align__(16) unsigned char smem_raw[];
-    SgSmem &S = *reinterpret_cast<SgSmem *>(smem_raw);
-    sg_clear(S);
+    __shared__ SgPriv P;
+    sgp_clear(P);
     __syncthreads();
-    // cache the gathered orders fields of the last looked-up row
-    unsigned int last = kNoRow;
-    long long entry = 0;
-    int carrier = -1, cnt = 0;
-    probe_rows(ol_w, ol_d, ol_o, ol_dl, n, jo, [&](unsigned int row, long long dl) {
-        if (row == kNoRow) return;  // inner join: orphan lines drop out
-        if (row != last) {
-            last = row;
-            entry = __ldg(oc.entry + row);
-            carrier = __ldg(oc.carrier + row);
-            cnt = __ldg(oc.cnt + row);
+    probe_rows4(ol_w, ol_d, ol_o, ol_dl, n, jo, [&](const unsigned int (&r)[4], const long long (&dl)[4], bool) {
+        // gathers of the distinct looked-up rows (independent loads)
+        long long entry[4];
+        int carrier[4], cnt[4];
+#pragma unroll
+        for (int j = 0; j < 4; ++j) {
+            if (r[j] != kNoRow && (j == 0 || r[j] != r[j - 1])) {
+                entry[j] = __ldg(oc.entry + r[j]);
+                carrier[j] = __ldg(oc.carrier + r[j]);
+                cnt[j] = __ldg(oc.cnt + r[j]);
+            } else if (j > 0) {
+                entry[j] = entry[j - 1]; carrier[j] = carrier[j - 1]; cnt[j] = cnt[j - 1];
+            } else {
+                entry[j] = 0; carrier[j] = -1; cnt[j] = 0;
+            }
         }
-        // o_entry_d <= ol_delivery_d AND ol_delivery_d < d_hi; NULL delivery -> UNKNOWN (R5)
-        if (dl == kNullTs || dl < entry || dl >= d_hi) return;
-        // carrier = 1 OR carrier = 2 / carrier <> 1 AND carrier <> 2; NULL (-1) -> neither
-        const unsigned hi = (carrier == 1) | (carrier == 2);
-        const unsigned lo = (carrier != -1) & !hi;
-        sg_add(S, g, cnt, hi, lo);
+#pragma unroll
+        for (int j = 0; j < 4; ++j) {
+            // inner join (orphan lines drop out); o_entry_d <= ol_delivery_d AND
+            // ol_delivery_d < d_hi, a NULL delivery date is UNKNOWN (R5)
+            if (r[j] == kNoRow || dl[j] == kNullTs || dl[j] < entry[j] || dl[j] >= d_hi) continue;
+            // carrier = 1 OR carrier = 2 / carrier <> 1 AND carrier <> 2; NULL (-1) -> neither
+            const bool hi = (carrier[j] == 1) | (carrier[j] == 2);
+            const bool lo = (carrier[j] != -1) & !hi;
+            sgp_add(P, g, cnt[j], hi, lo);
+        }
     });
-    sg_flush(S, g);
+    sgp_flush(P, g);
 }
 
 __global__ void __launch_bounds__(kThreads)
@@ -260,26 +319,32 @@ q4_mark_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ ol_
                const int32_t *__restrict__ ol_o, const int64_t *__restrict__ ol_dl, uint64_t n,
                JoinIndex jo, const int64_t *__restrict__ o_entry, long long e_lo, long long e_hi,
                uint8_t *mark) {
-    unsigned int last = kNoRow;
-    long long entry = 0;
-    probe_rows(ol_w, ol_d, ol_o, ol_dl, n, jo, [&](unsigned int row, long long dl) {
-        if (row == kNoRow) return;
-        if (row != last) { last = row; entry = __ldg(o_entry + row); }
-        // the order is in the entry window and this line has ol_delivery_d >= o_entry_d
-        if (entry >= e_lo && entry < e_hi && dl != kNullTs && dl >= entry) mark[row] = 1;
+    probe_rows4(ol_w, ol_d, ol_o, ol_dl, n, jo, [&](const unsigned int (&r)[4], const long long (&dl)[4], bool) {
+        long long entry[4];
+#pragma unroll
+        for (int j = 0; j < 4; ++j)
+            entry[j] = (r[j] != kNoRow && (j == 0 || r[j] != r[j - 1])) ? __ldg(o_entry + r[j])
+                       : (j > 0 ? entry[j - 1] : 0);
+#pragma unroll
+        for (int j = 0; j < 4; ++j)
+            // the order is in the entry window and this line has ol_delivery_d >= o_entry_d
+            if (r[j] != kNoRow && entry[j] >= e_lo && entry[j] < e_hi && dl[j] != kNullTs && dl[j] >= entry[j])
+                mark[r[j]] = 1;
     });
 }
 
 __global__ void __launch_bounds__(kThreads)
 q4_count_kernel(const uint8_t *__restrict__ mark, const int32_t *__restrict__ o_cnt, uint64_t n,
                 SmallGroups g) {
-    extern __shared__ __align__(16) unsigned char smem_raw[];
-    SgSmem &S = *reinterpret_cast<SgSmem *>(smem_raw);
+    __shared__ SgSmem S;
     sg_clear(S);
     __syncthreads();
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
-         i += (uint64_t)gridDim.x * blockDim.x)
-        if (mark[i]) sg_add(S, g, __ldg(o_cnt + i), 1u, 0u);
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    for (uint64_t b = (uint64_t)blockIdx.x * blockDim.x + (threadIdx.x & ~31u); b < n; b += stride) {
+        const uint64_t i = b + (threadIdx.x & 31);  // warp-uniform loop
+        const bool ok = i < n && mark[i];
+        sg_warp_add(S, g, ok, ok ? __ldg(o_cnt + i) : 0, true, false);
+    }
     sg_flush(S, g);
 }
 
@@ -404,13 +469,8 @@ void launch_jx_build_orders(const int32_t *o_w, const int32_t *o_d, const int32_
 void launch_q12_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o, const int64_t *ol_dl,
                       uint64_t n_ol, const JoinIndex &jo, const int64_t *o_entry, const int32_t *o_carrier,
                       const int32_t *o_cnt, int64_t d_hi, const SmallGroups &g, int num_sms, cudaStream_t st) {
-    static bool attr = false;
-    if (!attr) {
-        cudaFuncSetAttribute(q12_probe_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(SgSmem));
-        attr = true;
-    }
-    const unsigned grid = grid_for((n_ol + 3) / 4, kThreads, num_sms, 4);
-    q12_probe_kernel<<<grid, kThreads, sizeof(SgSmem), st>>>(ol_w, ol_d, ol_o, ol_dl, n_ol, jo,
+    const unsigned grid = grid_for((n_ol + 3) / 4, kThreads, num_sms, 8);
+    q12_probe_kernel<<<grid, kThreads, 0, st>>>(ol_w, ol_d, ol_o, ol_dl, n_ol, jo,
                                                              OrderCols{o_entry, o_carrier, o_cnt}, d_hi, g);
     count_launches(1);
 }
@@ -419,11 +479,6 @@ void launch_q4(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o, co
                uint64_t n_ol, const JoinIndex &jo, const int64_t *o_entry, const int32_t *o_cnt,
                uint64_t n_o, int64_t e_lo, int64_t e_hi, uint8_t *mark, const SmallGroups &g,
                int num_sms, cudaStream_t st, PhaseMarks *marks) {
-    static bool attr = false;
-    if (!attr) {
-        cudaFuncSetAttribute(q4_count_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(SgSmem));
-        attr = true;
-    }
     if (marks) marks->begin("q4_semijoin_mark");
     if (n_ol)
         q4_mark_kernel<<<grid_for((n_ol + 3) / 4, kThreads, num_sms, 8), kThreads, 0, st>>>(
@@ -431,7 +486,7 @@ void launch_q4(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o, co
     if (marks) marks->end();
     if (marks) marks->begin("q4_count");
     if (n_o)
-        q4_count_kernel<<<grid_for(n_o, kThreads, num_sms, 4), kThreads, sizeof(SgSmem), st>>>(mark, o_cnt, n_o, g);
+        q4_count_kernel<<<grid_for(n_o, kThreads, num_sms, 8), kThreads, 0, st>>>(mark, o_cnt, n_o, g);
     if (marks) marks->end();
     count_launches((n_ol ? 1 : 0) + (n_o ? 1 : 0));
 }
@@ -453,7 +508,8 @@ void launch_q14(const int64_t *deliv, const int32_t *i_id, const int64_t *amt, u
         cudaFuncSetAttribute(q14_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, kQ14SmemWords * 4);
         attr = true;
     }
-    const int per_sm = smem_map ? (m.words * 4 > 48 * 1024 ? 2 : 4) : 8;
+    // 4 blocks per SM (each copies the map into shared memory; more blocks measured slower)
+    const int per_sm = smem_map ? (m.words * 4 > (48u << 10) ? 2 : 4) : 8;
     const unsigned grid = grid_for((n + 3) / 4, kThreads, num_sms, per_sm);
     const auto *D = reinterpret_cast<const longlong2 *>(deliv);
     const auto *I = reinterpret_cast<const int4 *>(i_id);

@@ -128,12 +128,21 @@ __device__ __forceinline__ void probe_lane_group(const Q18Scratch &s, const Key3
         unsigned carry_c = __shfl_up_sync(kFull, ic, 1);
         if (!cont) { carry_s = 0; carry_c = 0; }
         if (!valid) return;
-        // runs ending inside the lane (rows 0..2): the first run also gets the carry
-        if (b1) flush_run(s, k[0], s0 + carry_s, c0 + carry_c);
-        if (b2) flush_run(s, k[1], s1 + (b1 ? 0 : carry_s), c1 + (b1 ? 0 : carry_c));
-        if (b3) flush_run(s, k[2], s2 + ((b1 | b2) ? 0 : carry_s), c2 + ((b1 | b2) ? 0 : carry_c));
-        // the lane's last run ends here unless the next lane continues it
-        if (!next_cont) flush_run(s, k[3], is, ic);
+        // runs ending inside the lane (rows 0..2; the first run also gets the carry) and the
+        // lane's last run unless the next lane continues it: all lookups are issued first
+        // (independent loads in flight together), then the atomics
+        const bool f[4] = {b1, b2, b3, !next_cont};
+        const long long fs[4] = {s0 + carry_s, s1 + (b1 ? 0 : carry_s), s2 + ((b1 | b2) ? 0 : carry_s), is};
+        const unsigned fc[4] = {c0 + carry_c, c1 + (b1 ? 0 : carry_c), c2 + ((b1 | b2) ? 0 : carry_c), ic};
+        unsigned int row[4];
+#pragma unroll
+        for (int j = 0; j < 4; ++j) row[j] = f[j] ? jx_lookup(s.jo, k[j].w, k[j].d, k[j].o) : kNoRow;
+#pragma unroll
+        for (int j = 0; j < 4; ++j)
+            if (row[j] != kNoRow) {
+                atomicAdd(reinterpret_cast<unsigned long long *>(&s.acc[row[j]].sum), (unsigned long long)fs[j]);
+                atomicAdd(&s.acc[row[j]].cnt, fc[j]);
+            }
 }
 
 __global__ void __launch_bounds__(kProbeThreads)
