@@ -39,7 +39,7 @@ __all__ = [
     "DAY_US", "ts_us", "generate", "generate_item", "neworder_delta",
     "warehouse_ranges", "concat_tables", "TABLE_COLUMNS", "NewOrderState", "neworder_batch",
     "ROW_DTYPES", "to_records", "DeliveryState", "delivery_inputs", "delivery_batch",
-    "i_data_prefix2",
+    "i_data_prefix2", "prefix2",
 ]
 
 
@@ -65,7 +65,8 @@ TABLE_COLUMNS = {
                ("o_c_id", np.int32), ("o_ol_cnt", np.int32), ("o_carrier_id", np.int32),
                ("o_all_local", np.int32), ("o_entry_d", np.int64)],
     "customer": [("c_w_id", np.int32), ("c_d_id", np.int32), ("c_id", np.int32),
-                 ("c_last", np.int32)],
+                 ("c_last", np.int32), ("c_state", "S2"), ("c_state_p2", np.int32)],
+    "new_order": [("no_w_id", np.int32), ("no_d_id", np.int32), ("no_o_id", np.int32)],
     "item": [("i_id", np.int32), ("i_price", np.int64), ("i_data", "S50"), ("i_data_p2", np.int32)],
 }
 
@@ -145,6 +146,10 @@ def _warehouse(w: int, seed: int, mode: str, sc: Scale):
     b = rng.integers(0, 1000, size=D * C, dtype=np.int32)
     nurand = ((a | b) + NURAND_C_LAST) % 1000
     c_last = np.where(c_id <= 1000, c_id - 1, nurand).astype(np.int32)
+    # c_state: random a-string of 2 characters (TPC-C 4.3.3.1 [EXT]) over the same alphabet as
+    # i_data; drawn LAST from the warehouse stream so that every earlier column is unchanged
+    st = ALNUM[rng.integers(0, len(ALNUM), size=(D * C, 2))]
+    c_state = np.ascontiguousarray(st).view("S2").reshape(D * C)
 
     wi = np.int32(w)
     ol = {
@@ -160,17 +165,30 @@ def _warehouse(w: int, seed: int, mode: str, sc: Scale):
         "o_all_local": np.ones(n_o, dtype=np.int32), "o_entry_d": o_entry,
     }
     customer = {"c_w_id": np.full(D * C, wi, dtype=np.int32), "c_d_id": c_d, "c_id": c_id,
-                "c_last": c_last}
-    return {"order_line": ol, "orders": orders, "customer": customer}
+                "c_last": c_last, "c_state": c_state, "c_state_p2": prefix2(c_state)}
+    # new_order: one row per undelivered order (TPC-C 4.3.3.1: the last 900 orders of each
+    # district, NO_O_ID 2101..3000), in (d, o_id) order
+    und = o_carrier == -1
+    new_order = {"no_w_id": np.full(int(und.sum()), wi, dtype=np.int32), "no_d_id": o_d[und],
+                 "no_o_id": o_id[und]}
+    return {"order_line": ol, "orders": orders, "customer": customer, "new_order": new_order}
 
 
 ALNUM = np.frombuffer(b"abcdefghijklmnopqrstuvwxyzABCDEFGHIJKLMNOPQRSTUVWXYZ0123456789", np.uint8)
 
 
-def i_data_prefix2(i_data) -> np.ndarray:
-    """(byte0 << 8) | byte1 of each string (0 for a missing byte)."""
-    b = np.frombuffer(np.asarray(i_data, dtype="S50").tobytes(), np.uint8).reshape(-1, 50)
+def prefix2(strings) -> np.ndarray:
+    """(byte0 << 8) | byte1 of each fixed-width byte string (0 for a missing byte): the device
+    encoding of a string column's first two characters (R29)."""
+    a = np.asarray(strings)
+    width = max(a.dtype.itemsize, 2)
+    b = np.frombuffer(a.astype(f"S{width}").tobytes(), np.uint8).reshape(-1, width)
     return ((b[:, 0].astype(np.int32) << 8) | b[:, 1].astype(np.int32)).astype(np.int32)
+
+
+def i_data_prefix2(i_data) -> np.ndarray:
+    """(byte0 << 8) | byte1 of each i_data string (0 for a missing byte)."""
+    return prefix2(np.asarray(i_data, dtype="S50"))
 
 
 def generate_item(seed: int = 1, scale: Scale = FULL):
@@ -282,8 +300,16 @@ def neworder_delta(state: NewOrderState, n_txn: int, *, seed: int, batch: int,
                          ("ol_quantity", q), ("ol_amount", q * int(item["i_price"][i - 1]))):
                 cols_l[k].append(v)
     dts = {c: dt for t in ("orders", "order_line") for c, dt in TABLE_COLUMNS[t]}
-    return {"orders": {k: np.asarray(v, dtype=dts[k]) for k, v in cols_o.items()},
-            "order_line": {k: np.asarray(v, dtype=dts[k]) for k, v in cols_l.items()}}
+    orders = {k: np.asarray(v, dtype=dts[k]) for k, v in cols_o.items()}
+    return {"orders": orders,
+            "order_line": {k: np.asarray(v, dtype=dts[k]) for k, v in cols_l.items()},
+            "new_order": _new_order_rows(orders)}
+
+
+def _new_order_rows(orders: dict) -> dict:
+    """The new_order rows a NewOrder transaction inserts: one per new order (TPC-C 2.4.2.2)."""
+    return {"no_w_id": orders["o_w_id"].astype(np.int32), "no_d_id": orders["o_d_id"].astype(np.int32),
+            "no_o_id": orders["o_id"].astype(np.int32)}
 
 
 def neworder_batch(state: NewOrderState, n_txn: int, *, seed: int, batch: int, item=None):
@@ -330,7 +356,7 @@ def neworder_batch(state: NewOrderState, n_txn: int, *, seed: int, batch: int, i
           "ol_o_id": np.repeat(o_id.astype(np.int32), cnt), "ol_number": number, "ol_i_id": iid,
           "ol_supply_w_id": np.repeat(w, cnt), "ol_delivery_d": np.full(n_ol, NULL_TS, np.int64),
           "ol_quantity": qty, "ol_amount": amount}
-    return {"orders": orders, "order_line": ol}
+    return {"orders": orders, "order_line": ol, "new_order": _new_order_rows(orders)}
 
 
 # NSM record layouts of the host row store (one record per row, fields in schema order)

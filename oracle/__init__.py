@@ -1,4 +1,4 @@
-"""CPU oracle for CH-benCHmark Q1 / Q6 / Q18 (and NEXT-2: Q14 / Q12 / Q4) — TEST INFRASTRUCTURE ONLY.
+"""CPU oracle for CH-benCHmark Q1 / Q6 / Q18 (and NEXT-2: Q14 / Q12 / Q4 / Q3) — TEST INFRASTRUCTURE ONLY.
 
 Only ``tests/``, ``__graft_entry__.smoke()`` and ``bench.py`` (its ``cpu_baseline``
 leg and ``--impl reference``) may import this package. The product path
@@ -58,7 +58,11 @@ class _I(C.Structure):
 
 class _C(C.Structure):
     _fields_ = [("n", C.c_int64), ("w_id", C.c_void_p), ("d_id", C.c_void_p), ("c_id", C.c_void_p),
-                ("c_last", C.c_void_p)]
+                ("c_last", C.c_void_p), ("state", C.c_void_p), ("state_width", C.c_int64)]
+
+
+class _NO(C.Structure):
+    _fields_ = [("n", C.c_int64), ("w_id", C.c_void_p), ("d_id", C.c_void_p), ("o_id", C.c_void_p)]
 
 
 _lib = None
@@ -74,6 +78,7 @@ def _load():
         lib.oracle_q14.restype = C.c_int
         lib.oracle_q12.restype = C.c_int64
         lib.oracle_q4.restype = C.c_int64
+        lib.oracle_q3.restype = C.c_int64
         _lib = lib
     return _lib
 
@@ -164,7 +169,7 @@ def q18(tables, having):
     o, c = tables["orders"], tables["customer"]
     os_ = _o_struct(o, keep)
     cs = _C(len(c["c_w_id"]), keep(_col(c, "c_w_id", np.int32)), keep(_col(c, "c_d_id", np.int32)),
-            keep(_col(c, "c_id", np.int32)), keep(_col(c, "c_last", np.int32)))
+            keep(_col(c, "c_id", np.int32)), keep(_col(c, "c_last", np.int32)), None, 0)
     cap = max(1, len(o["o_w_id"]))
     while True:
         out = {k: np.zeros(cap, dt) for k, dt in Q18_COLUMNS}
@@ -238,3 +243,30 @@ def q4(tables, e_lo, e_hi):
     return _small_groups(lambda cap, *ps: lib.oracle_q4(C.byref(o), C.byref(ol), C.c_int64(e_lo),
                                                         C.c_int64(e_hi), C.c_int64(cap), *ps),
                          ["o_ol_cnt", "order_count"], [np.int32, np.int64])
+
+
+Q3_COLUMNS = [("ol_o_id", np.int32), ("ol_w_id", np.int32), ("ol_d_id", np.int32),
+              ("revenue", np.int64), ("o_entry_d", np.int64)]
+
+
+def q3(tables, entry_lo, prefix=b"A"):
+    """CH Q3 (customer ⋈ new_order ⋈ orders ⋈ order_line, GROUP BY, ORDER BY revenue DESC,
+    o_entry_d). Returns numpy columns ol_o_id, ol_w_id, ol_d_id, revenue, o_entry_d in order."""
+    lib, keep = _load(), _Keep()
+    ol = _ol_struct(tables["order_line"], keep)
+    os_ = _o_struct(tables["orders"], keep)
+    c, no = tables["customer"], tables["new_order"]
+    state = np.ascontiguousarray(np.asarray(c["c_state"], dtype="S2"))
+    cs = _C(len(c["c_w_id"]), keep(_col(c, "c_w_id", np.int32)), keep(_col(c, "c_d_id", np.int32)),
+            keep(_col(c, "c_id", np.int32)), None, keep(state), 2)
+    ns = _NO(len(no["no_w_id"]), keep(_col(no, "no_w_id", np.int32)),
+             keep(_col(no, "no_d_id", np.int32)), keep(_col(no, "no_o_id", np.int32)))
+    cap = max(1, len(no["no_w_id"]))
+    while True:
+        out = {k: np.zeros(cap, dt) for k, dt in Q3_COLUMNS}
+        n = lib.oracle_q3(C.byref(cs), C.byref(ns), C.byref(os_), C.byref(ol), C.c_int64(entry_lo),
+                          C.c_char_p(bytes(prefix)), C.c_int64(cap), *[_p(out[k]) for k, _ in Q3_COLUMNS])
+        _check(n if n < 0 else 0)
+        if n <= cap:
+            return {k: v[:n] for k, v in out.items()}
+        cap = n

@@ -434,3 +434,99 @@ done:
     map_free(&hl); map_free(&hg);
     return st == OR_OK ? ng : st;
 }
+
+/* ----------------------------------------------------------------- CH Q3 -- */
+/* GROUP BY ol_o_id, ol_w_id, ol_d_id, o_entry_d */
+enum { G3_O_ID, G3_W_ID, G3_D_ID, G3_ENTRY_D, G3_NKEY };
+typedef struct { int64_t key[G3_NKEY]; int64_t revenue; } q3_group;
+
+static int cmp_q3(const void *pa, const void *pb) {
+    const q3_group *a = pa, *b = pb;
+    int c;
+    if ((c = cmp_i64(b->revenue, a->revenue))) return c;                     /* revenue DESC */
+    if ((c = cmp_i64(a->key[G3_ENTRY_D], b->key[G3_ENTRY_D]))) return c;      /* o_entry_d ASC */
+    static const int tie[] = {G3_W_ID, G3_D_ID, G3_O_ID};                     /* R33 */
+    for (int i = 0; i < 3; i++)
+        if ((c = cmp_i64(a->key[tie[i]], b->key[tie[i]]))) return c;
+    return 0;
+}
+
+int64_t oracle_q3(const or_customer *c, const or_new_order *no, const or_orders *o,
+                  const or_order_line *ol, int64_t entry_lo, const char *prefix, int64_t cap,
+                  int32_t *ol_o_id, int32_t *ol_w_id, int32_t *ol_d_id, int64_t *revenue,
+                  int64_t *o_entry_d) {
+    ormap hc, hn, ho, hg;
+    int st = OR_OK;
+    int64_t ngroups = 0, gcap = 1024;
+    q3_group *g = NULL;
+    memset(&hc, 0, sizeof hc); memset(&hn, 0, sizeof hn);
+    memset(&ho, 0, sizeof ho); memset(&hg, 0, sizeof hg);
+    if (map_init(&hc, 3, c->n) || map_init(&hn, 3, no->n) || map_init(&ho, 3, o->n) ||
+        map_init(&hg, G3_NKEY, 1024)) { st = OR_NOMEM; goto done; }
+    g = malloc(sizeof(q3_group) * gcap);
+    if (!g) { st = OR_NOMEM; goto done; }
+    /* join indexes (multimaps, every row inserted): customer (c_w_id, c_d_id, c_id),
+     * new_order (no_w_id, no_d_id, no_o_id), orders (o_w_id, o_d_id, o_id) */
+    for (int64_t r = 0; r < c->n; r++) {
+        int64_t k[3] = {c->w_id[r], c->d_id[r], c->c_id[r]};
+        if (map_append(&hc, k, r) < 0) { st = OR_NOMEM; goto done; }
+    }
+    for (int64_t r = 0; r < no->n; r++) {
+        int64_t k[3] = {no->w_id[r], no->d_id[r], no->o_id[r]};
+        if (map_append(&hn, k, r) < 0) { st = OR_NOMEM; goto done; }
+    }
+    for (int64_t r = 0; r < o->n; r++) {
+        int64_t k[3] = {o->w_id[r], o->d_id[r], o->o_id[r]};
+        if (map_append(&ho, k, r) < 0) { st = OR_NOMEM; goto done; }
+    }
+    /* scan order_line; ol = o on (w, d, o_id); o_entry_d > entry_lo; no = o on (w, d, o_id);
+     * c = o on (w, d, c_id) with c_state LIKE 'prefix%'; one joined tuple per combination */
+    for (int64_t l = 0; l < ol->n; l++) {
+        int64_t ko[3] = {ol->w_id[l], ol->d_id[l], ol->o_id[l]};
+        for (int64_t eo = map_first(&ho, ko); eo >= 0; eo = map_next_same(&ho, eo, ko)) {
+            int64_t orow = ho.val[eo];
+            if (ts_gt(o->entry_d[orow], entry_lo) != SQL_TRUE) continue;
+            int64_t kn[3] = {o->w_id[orow], o->d_id[orow], o->o_id[orow]};
+            for (int64_t en = map_first(&hn, kn); en >= 0; en = map_next_same(&hn, en, kn)) {
+                int64_t kc[3] = {o->w_id[orow], o->d_id[orow], o->c_id[orow]};
+                for (int64_t ec = map_first(&hc, kc); ec >= 0; ec = map_next_same(&hc, ec, kc)) {
+                    int64_t crow = hc.val[ec];
+                    if (!like_prefix(c->state + crow * c->state_width, c->state_width, prefix)) continue;
+                    int64_t gk[G3_NKEY];
+                    gk[G3_O_ID] = ol->o_id[l]; gk[G3_W_ID] = ol->w_id[l]; gk[G3_D_ID] = ol->d_id[l];
+                    gk[G3_ENTRY_D] = o->entry_d[orow];
+                    int64_t eg = map_first(&hg, gk), gi;
+                    if (eg < 0) {
+                        if (ngroups == gcap) {
+                            gcap *= 2;
+                            q3_group *ng = realloc(g, sizeof(q3_group) * gcap);
+                            if (!ng) { st = OR_NOMEM; goto done; }
+                            g = ng;
+                        }
+                        gi = ngroups++;
+                        memcpy(g[gi].key, gk, sizeof gk);
+                        g[gi].revenue = 0;
+                        if (map_append(&hg, gk, gi) < 0) { st = OR_NOMEM; goto done; }
+                    } else {
+                        gi = hg.val[eg];
+                    }
+                    if (__builtin_add_overflow(g[gi].revenue, ol->amount[l], &g[gi].revenue)) {
+                        st = OR_OVERFLOW; goto done;
+                    }
+                }
+            }
+        }
+    }
+    qsort(g, (size_t)ngroups, sizeof(q3_group), cmp_q3);               /* ORDER BY */
+    for (int64_t i = 0; i < ngroups && i < cap; i++) {
+        ol_o_id[i] = (int32_t)g[i].key[G3_O_ID];
+        ol_w_id[i] = (int32_t)g[i].key[G3_W_ID];
+        ol_d_id[i] = (int32_t)g[i].key[G3_D_ID];
+        revenue[i] = g[i].revenue;
+        o_entry_d[i] = g[i].key[G3_ENTRY_D];
+    }
+done:
+    free(g);
+    map_free(&hc); map_free(&hn); map_free(&ho); map_free(&hg);
+    return st == OR_OK ? ngroups : st;
+}

@@ -6,7 +6,7 @@
  * CUDA path (paper_conf_cidr_appuswamykpa17_b200/, include/), and never includes them.
  *
  * What it computes: the plain SQL definitions of CH-benCHmark Q1, Q6 and Q18, and (NEXT-2)
- * Q14, Q12 and Q4
+ * Q14, Q12, Q4 and Q3
  * (SURVEY.md Appendix A.1 [EXT]; the paper's OLAP path is PAPER.md L524-572, its only
  * query text is "TPC-H Q6, a selection over the lineitem table", L687-688), evaluated
  * row at a time, single-threaded, with SQL three-valued logic for NULLs.
@@ -53,7 +53,14 @@ typedef struct {
 typedef struct {
     int64_t n;
     const int32_t *w_id, *d_id, *c_id, *c_last;
+    const char *state;              /* c_state: n strings of `state_width` bytes (Q3 only) */
+    int64_t state_width;
 } or_customer;
+
+typedef struct {
+    int64_t n;
+    const int32_t *w_id, *d_id, *o_id;  /* no_w_id, no_d_id, no_o_id */
+} or_new_order;
 
 /* Status codes. */
 #define OR_OK        0
@@ -109,6 +116,19 @@ int64_t oracle_q12(const or_orders *o, const or_order_line *ol, int64_t d_hi, in
  * GROUP BY o_ol_cnt ORDER BY o_ol_cnt. Writes min(ngroups, cap) rows; returns ngroups or < 0. */
 int64_t oracle_q4(const or_orders *o, const or_order_line *ol, int64_t e_lo, int64_t e_hi,
                   int64_t cap, int32_t *o_ol_cnt, int64_t *order_count);
+
+/* CH Q3: SELECT ol_o_id, ol_w_id, ol_d_id, SUM(ol_amount) AS revenue, o_entry_d
+ * FROM customer, new_order, orders, order_line
+ * WHERE c_state LIKE prefix || '%' AND c_id = o_c_id AND c_w_id = o_w_id AND c_d_id = o_d_id
+ *   AND no_w_id = o_w_id AND no_d_id = o_d_id AND no_o_id = o_id
+ *   AND ol_w_id = o_w_id AND ol_d_id = o_d_id AND ol_o_id = o_id AND o_entry_d > entry_lo
+ * GROUP BY ol_o_id, ol_w_id, ol_d_id, o_entry_d ORDER BY revenue DESC, o_entry_d
+ * (ties: ol_w_id, ol_d_id, ol_o_id ASC, R33). Output columns ol_o_id, ol_w_id,
+ * ol_d_id, revenue, o_entry_d. Writes min(nrows, cap) rows; returns nrows or < 0. */
+int64_t oracle_q3(const or_customer *c, const or_new_order *no, const or_orders *o,
+                  const or_order_line *ol, int64_t entry_lo, const char *prefix, int64_t cap,
+                  int32_t *ol_o_id, int32_t *ol_w_id, int32_t *ol_d_id, int64_t *revenue,
+                  int64_t *o_entry_d);
 
 #ifdef __cplusplus
 }

@@ -68,6 +68,16 @@ def sqlite_load(tables):
         db.executemany("INSERT INTO item VALUES (?,?)",
                        zip(it["i_id"].tolist(), [bytes(x).decode("latin-1") for x in it["i_data"]]))
         db.execute("CREATE INDEX ii ON item (i_id)")
+    if "c_state" in c:
+        db.execute("ALTER TABLE customer ADD COLUMN c_state TEXT")
+        db.executemany("UPDATE customer SET c_state = ? WHERE rowid = ?",
+                       [(bytes(x).decode("latin-1"), i + 1) for i, x in enumerate(c["c_state"])])
+    if "new_order" in tables:
+        no = tables["new_order"]
+        db.execute("CREATE TABLE new_order (no_w_id INT, no_d_id INT, no_o_id INT)")
+        db.executemany("INSERT INTO new_order VALUES (?,?,?)",
+                       zip(no["no_w_id"].tolist(), no["no_d_id"].tolist(), no["no_o_id"].tolist()))
+        db.execute("CREATE INDEX ino ON new_order (no_w_id, no_d_id, no_o_id)")
     db.execute("PRAGMA case_sensitive_like = ON")  # SQL LIKE is case-sensitive
     return db
 
@@ -125,6 +135,18 @@ def sqlite_q4(db, e_lo, e_hi):
         "WHERE o_entry_d >= ? AND o_entry_d < ? AND EXISTS (SELECT * FROM order_line"
         " WHERE o_id = ol_o_id AND o_w_id = ol_w_id AND o_d_id = ol_d_id AND ol_delivery_d >= o_entry_d) "
         "GROUP BY o_ol_cnt ORDER BY o_ol_cnt", (e_lo, e_hi)).fetchall()
+
+
+def sqlite_q3(db, entry_lo, prefix="A"):
+    """CH Q3 verbatim (timestamp literal as int64 us)."""
+    return db.execute(
+        "SELECT ol_o_id, ol_w_id, ol_d_id, SUM(ol_amount) AS revenue, o_entry_d "
+        "FROM customer, new_order, orders, order_line "
+        "WHERE c_state LIKE ? AND c_id = o_c_id AND c_w_id = o_w_id AND c_d_id = o_d_id "
+        "  AND no_w_id = o_w_id AND no_d_id = o_d_id AND no_o_id = o_id "
+        "  AND ol_w_id = o_w_id AND ol_d_id = o_d_id AND ol_o_id = o_id AND o_entry_d > ? "
+        "GROUP BY ol_o_id, ol_w_id, ol_d_id, o_entry_d ORDER BY revenue DESC, o_entry_d",
+        (prefix + "%", entry_lo)).fetchall()
 
 
 def sqlite_delivery(db, w, carrier, ts, districts):
@@ -195,6 +217,29 @@ def brute_q18(tables, having):
             groups[k] = groups.get(k, 0) + la
     out = [(k[4], k[3], k[0], k[5], k[6], s, k[1], k[2]) for k, s in groups.items() if s > having]
     out.sort(key=lambda r: (-r[5], r[3], r[6], r[7], r[2], r[1], r[0], r[4]))
+    return out
+
+
+def brute_q3(tables, entry_lo, prefix=b"A"):
+    """CH Q3's WHERE over the cartesian product customer x new_order x orders x order_line,
+    the conjunction evaluated in two stages (conjuncts without order_line first, over
+    customer x new_order x orders; then the order_line conjuncts over that x order_line)."""
+    C = list(zip(tables["customer"]["c_w_id"].tolist(), tables["customer"]["c_d_id"].tolist(),
+                 tables["customer"]["c_id"].tolist(), [bytes(x) for x in tables["customer"]["c_state"]]))
+    NO = _rows(tables["new_order"], ["no_w_id", "no_d_id", "no_o_id"])
+    O = _rows(tables["orders"], ["o_w_id", "o_d_id", "o_id", "o_c_id", "o_entry_d"])
+    L = _rows(tables["order_line"], ["ol_w_id", "ol_d_id", "ol_o_id", "ol_amount"])
+    stage = [(ow, od, oid, oent)
+             for (cw, cd, cid, cst), (nw, nd, no), (ow, od, oid, ocid, oent) in itertools.product(C, NO, O)
+             if cst.startswith(prefix) and cid == ocid and cw == ow and cd == od
+             and nw == ow and nd == od and no == oid and oent > entry_lo]
+    groups = {}
+    for (ow, od, oid, oent), (lw, ld, lo, la) in itertools.product(stage, L):
+        if lw == ow and ld == od and lo == oid:
+            k = (lo, lw, ld, oent)
+            groups[k] = groups.get(k, 0) + la
+    out = [(k[0], k[1], k[2], s, k[3]) for k, s in groups.items()]
+    out.sort(key=lambda r: (-r[3], r[4], r[1], r[2], r[0]))
     return out
 
 
@@ -317,3 +362,37 @@ def golden_next2(name="ch_next2.json"):
     params = {"q14": (iso_us(p["q14"][0]), iso_us(p["q14"][1]), p["q14"][2].encode()),
               "q12": (iso_us(p["q12"][0]),), "q4": (iso_us(p["q4"][0]), iso_us(p["q4"][1]))}
     return tables, params, g["expected"]
+
+
+def golden_q3(name="ch_q3.json"):
+    """The CH Q3 fixture as generator-shaped tables (+ params and expected rows)."""
+    with open(os.path.join(GOLDEN, name)) as f:
+        g = json.load(f)
+    tables = {}
+    for t in ("customer", "orders", "new_order", "order_line"):
+        cols, rows = g[t]["columns"], g[t]["rows"]
+        tab = {}
+        for j, c in enumerate(cols):
+            vals = [r[j] for r in rows]
+            if c == "o_entry_d":
+                tab[c] = np.array([iso_us(v) for v in vals], np.int64)
+            elif c == "ol_amount":
+                tab[c] = np.array(vals, np.int64)
+            elif c == "c_state":
+                tab[c] = np.array([v.encode() for v in vals], dtype="S2")
+            else:
+                tab[c] = np.array(vals, np.int32)
+        tables[t] = tab
+    c = tables["customer"]
+    b = np.frombuffer(c["c_state"].tobytes(), np.uint8).reshape(-1, 2)
+    c["c_state_p2"] = ((b[:, 0].astype(np.int32) << 8) | b[:, 1]).astype(np.int32)
+    ol = tables["order_line"]
+    n = len(ol["ol_w_id"])
+    ol["ol_delivery_d"] = np.full(n, NULL_SENTINEL, np.int64)
+    ol["ol_quantity"] = np.ones(n, np.int32)
+    ol["ol_i_id"] = np.ones(n, np.int32)
+    ol["ol_supply_w_id"] = ol["ol_w_id"].copy()
+    tables["orders"]["o_all_local"] = np.ones(len(tables["orders"]["o_id"]), np.int32)
+    p = g["params"]["q3"]
+    want = [(r[0], r[1], r[2], r[3], iso_us(r[4])) for r in g["expected"]["q3"]]
+    return tables, (iso_us(p[0]), p[1].encode()), want

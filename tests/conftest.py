@@ -8,6 +8,14 @@ if ROOT not in sys.path:
     sys.path.insert(0, ROOT)
 
 
+def pytest_sessionstart(session):
+    """Build libh2tap.so (nvcc, sm_100a) and the oracle checker in-tree before any test imports
+    the package: a fresh checkout has neither, and the package refuses to import without its
+    library (no CPU fallback). A no-op when both are up to date."""
+    import __graft_entry__
+    __graft_entry__.build()
+
+
 def pytest_configure(config):
     config.addinivalue_line("markers", "gpu: needs a B200 (runs the CUDA path through the C ABI)")
     config.addinivalue_line("markers", "slow: larger CPU cases")

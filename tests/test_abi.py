@@ -10,8 +10,8 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 
 @pytest.fixture(scope="module")
 def h():
-    from paper_conf_cidr_appuswamykpa17_b200 import _build
-    _build.build()
+    import __graft_entry__
+    __graft_entry__.build()
     import paper_conf_cidr_appuswamykpa17_b200 as mod
     return mod
 

@@ -37,7 +37,8 @@ def test_shards_are_byte_identical_slices(world):
     for lo, hi in chgen.warehouse_ranges(W, world):
         part = chgen.generate(lo, hi, seed=3, with_item=False)
         for tname, cols in part.items():
-            wcol = {"order_line": "ol_w_id", "orders": "o_w_id", "customer": "c_w_id"}[tname]
+            wcol = {"order_line": "ol_w_id", "orders": "o_w_id", "customer": "c_w_id",
+                    "new_order": "no_w_id"}[tname]
             m = (whole[tname][wcol] >= lo) & (whole[tname][wcol] < hi)
             for cname, arr in cols.items():
                 assert np.array_equal(arr, whole[tname][cname][m]), (tname, cname)
@@ -59,3 +60,22 @@ def test_neworder_delta_appends_fresh_orders():
     assert (d["orders"]["o_id"] >= 3001).all()
     assert len(d["order_line"]["ol_o_id"]) == int(d["orders"]["o_ol_cnt"].sum())
     assert (d["order_line"]["ol_delivery_d"] == chgen.NULL_TS).all()
+
+
+def test_new_order_and_c_state():
+    """new_order = the undelivered orders (TPC-C 4.3.3.1: o_id 2101..3000 per district, matching
+    orders with a NULL carrier, TPC-C consistency condition 5); c_state 2 characters of the
+    a-string alphabet, its device encoding = (byte0 << 8) | byte1; NewOrder deltas insert one
+    new_order row per order."""
+    t = chgen.generate(1, 3, seed=2)
+    o, no, c = t["orders"], t["new_order"], t["customer"]
+    assert len(no["no_o_id"]) == 2 * 10 * 900
+    und = o["o_carrier_id"] == -1
+    assert set(zip(no["no_w_id"].tolist(), no["no_d_id"].tolist(), no["no_o_id"].tolist())) == \
+        set(zip(o["o_w_id"][und].tolist(), o["o_d_id"][und].tolist(), o["o_id"][und].tolist()))
+    assert no["no_o_id"].min() == 2101 and no["no_o_id"].max() == 3000
+    st = [bytes(x) for x in c["c_state"]]
+    assert all(len(x) == 2 and x.isalnum() for x in st)
+    assert [x[0] << 8 | x[1] for x in st] == c["c_state_p2"].tolist()
+    d = chgen.neworder_batch(chgen.NewOrderState(1, 3), 7, seed=1, batch=0)
+    assert d["new_order"]["no_o_id"].tolist() == d["orders"]["o_id"].tolist()
