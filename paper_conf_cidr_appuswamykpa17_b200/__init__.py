@@ -33,9 +33,9 @@ H2TAP_ECUDA, H2TAP_ENCCL, H2TAP_EPLAN, H2TAP_EDUPKEY, H2TAP_ESHAPE = -4, -5, -6,
 STATUS_NAMES = {0: "OK", -1: "EINVAL", -2: "ESTALE", -3: "ENOMEM", -4: "ECUDA", -5: "ENCCL",
                 -6: "EPLAN", -7: "EDUPKEY", -8: "ESHAPE", -9: "EOVERFLOW"}
 H2TAP_I32, H2TAP_I64, H2TAP_F64 = 1, 2, 3
-H2TAP_T_ORDER_LINE, H2TAP_T_ORDERS, H2TAP_T_CUSTOMER, H2TAP_T_ITEM = 1, 2, 3, 4
+H2TAP_T_ORDER_LINE, H2TAP_T_ORDERS, H2TAP_T_CUSTOMER, H2TAP_T_ITEM, H2TAP_T_NEW_ORDER = 1, 2, 3, 4, 5
 H2TAP_Q1, H2TAP_Q6, H2TAP_Q18 = 1, 6, 18
-H2TAP_Q4, H2TAP_Q12, H2TAP_Q14 = 4, 12, 14  # NEXT-2 CH queries
+H2TAP_Q3, H2TAP_Q4, H2TAP_Q12, H2TAP_Q14 = 3, 4, 12, 14  # NEXT-2 CH queries
 H2TAP_FULL_RELOAD = 1
 H2TAP_LOAD_ASYNC = 1
 H2TAP_RESULT_DEVICE = 1
@@ -55,8 +55,10 @@ SCHEMA = {
         ("o_ol_cnt", H2TAP_I32), ("o_carrier_id", H2TAP_I32), ("o_all_local", H2TAP_I32),
         ("o_entry_d", H2TAP_I64)]),
     "customer": (H2TAP_T_CUSTOMER, [
-        ("c_w_id", H2TAP_I32), ("c_d_id", H2TAP_I32), ("c_id", H2TAP_I32), ("c_last", H2TAP_I32)]),
+        ("c_w_id", H2TAP_I32), ("c_d_id", H2TAP_I32), ("c_id", H2TAP_I32), ("c_last", H2TAP_I32),
+        ("c_state_p2", H2TAP_I32)]),
     "item": (H2TAP_T_ITEM, [("i_id", H2TAP_I32), ("i_price", H2TAP_I64), ("i_data_p2", H2TAP_I32)]),
+    "new_order": (H2TAP_T_NEW_ORDER, [("no_w_id", H2TAP_I32), ("no_d_id", H2TAP_I32), ("no_o_id", H2TAP_I32)]),
 }
 
 
@@ -482,6 +484,10 @@ def plan_columns():
                     "orders": ["o_w_id", "o_d_id", "o_id", "o_ol_cnt", "o_carrier_id", "o_entry_d"]},
         H2TAP_Q4: {"order_line": ["ol_w_id", "ol_d_id", "ol_o_id", "ol_delivery_d"],
                    "orders": ["o_w_id", "o_d_id", "o_id", "o_ol_cnt", "o_entry_d"]},
+        H2TAP_Q3: {"order_line": ["ol_w_id", "ol_d_id", "ol_o_id", "ol_amount"],
+                   "orders": ["o_w_id", "o_d_id", "o_id", "o_c_id", "o_ol_cnt", "o_entry_d"],
+                   "customer": ["c_w_id", "c_d_id", "c_id", "c_state_p2"],
+                   "new_order": ["no_w_id", "no_d_id", "no_o_id"]},
         H2TAP_Q6: {"order_line": ["ol_delivery_d", "ol_quantity", "ol_amount"]},
         H2TAP_Q1: {"order_line": ["ol_number", "ol_delivery_d", "ol_quantity", "ol_amount"]},
         H2TAP_Q18: {"order_line": ["ol_w_id", "ol_d_id", "ol_o_id", "ol_amount"],

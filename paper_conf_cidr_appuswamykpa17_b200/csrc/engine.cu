@@ -81,15 +81,16 @@ struct Fail {  // thrown internally, converted to a status at the ABI boundary
     } while (0)
 
 // ============================================================== schema ===
-constexpr int kTables = 5;  // index = table id (1..4)
+constexpr int kTables = 6;  // index = table id (1..5)
 constexpr int kMaxCols = 9;
-const int kNcols[kTables] = {0, 9, 8, 4, 3};
+const int kNcols[kTables] = {0, 9, 8, 5, 3, 3};
 const uint32_t kTypes[kTables][kMaxCols] = {
     {},
     {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64},
     {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64},
-    {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32},
-    {H2TAP_I32, H2TAP_I64, H2TAP_I32}};
+    {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32},
+    {H2TAP_I32, H2TAP_I64, H2TAP_I32},
+    {H2TAP_I32, H2TAP_I32, H2TAP_I32}};
 inline size_t type_size(uint32_t t) { return t == H2TAP_I32 ? 4 : 8; }
 constexpr uint64_t kPadRows = 64;  // over-allocation so 128-bit loads of the last tile stay in bounds
 
@@ -456,7 +457,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
     bool seen[kTables] = {};
     for (uint32_t i = 0; i < ntables; ++i) {
         const h2tap_table &t = tables[i];
-        if (t.table_id < 1 || t.table_id > 4) return fail(H2TAP_EINVAL, "unknown table id %u", t.table_id);
+        if (t.table_id < 1 || t.table_id >= (uint32_t)kTables) return fail(H2TAP_EINVAL, "unknown table id %u", t.table_id);
         if (seen[t.table_id]) return fail(H2TAP_EINVAL, "table %u listed twice", t.table_id);
         seen[t.table_id] = true;
         if (t.ncols == 0 || !t.cols) return fail(H2TAP_EINVAL, "table %u has no columns", t.table_id);
@@ -491,7 +492,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         uint32_t listed[kTables] = {};
         for (uint32_t i = 0; i < nupdates; ++i) {
             const h2tap_update &u = updates[i];
-            if (u.table_id < 1 || u.table_id > 4) return fail(H2TAP_EINVAL, "update %u: unknown table id %u", i, u.table_id);
+            if (u.table_id < 1 || u.table_id >= (uint32_t)kTables) return fail(H2TAP_EINVAL, "update %u: unknown table id %u", i, u.table_id);
             if (u.column_id >= (uint32_t)kNcols[u.table_id])
                 return fail(H2TAP_EINVAL, "update %u: unknown column id %u", i, u.column_id);
             if (u.type != kTypes[u.table_id][u.column_id])
@@ -934,6 +935,10 @@ JoinIndex plan_index(h2tap_engine *e, const View &v, int table, bool force_hash,
 }
 
 struct Q18Small { unsigned long long nout; unsigned int err, tie; Q18Stats st; };
+const char *const kQ18Names[8] = {"c_last", "c_id", "o_id", "o_entry_d", "o_ol_cnt", "amount_sum", "o_w_id", "o_d_id"};
+const uint32_t kQ18Types[8] = {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I32};
+const char *const kQ3Names[5] = {"ol_o_id", "ol_w_id", "ol_d_id", "revenue", "o_entry_d"};
+const uint32_t kQ3Types[5] = {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I64};
 
 void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     // a8: ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id, entirely on the device:
@@ -991,12 +996,11 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
                      &marks);
 }
 
-void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
-    const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
-    need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}, "Q18");
-    need_cols(v, O, {H2TAP_O_W_ID, H2TAP_O_D_ID, H2TAP_O_ID, H2TAP_O_C_ID, H2TAP_O_OL_CNT, H2TAP_O_ENTRY_D}, "Q18");
-    need_cols(v, C, {H2TAP_C_W_ID, H2TAP_C_D_ID, H2TAP_C_ID, H2TAP_C_LAST}, "Q18");
-    const uint64_t n_ol = v.n[OL], n_o = v.n[O], n_c = v.n[C];
+// Scratch of the orders/customer group-join (Q18, and Q3 which reuses it): join indexes,
+// per-orders-row accumulators, counters, statistics and the unsorted result rows (`rows_cap`).
+void q18_scratch(h2tap_engine *e, const View &v, QueryCtx &q, uint64_t rows_cap) {
+    const int O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
+    const uint64_t n_o = v.n[O];
     const bool force_hash = q.flags & H2TAP_QUERY_HASH_JOIN;
     Q18Scratch &s = q.q18;
     s.jo = plan_index(e, v, O, force_hash, "q18.jo");
@@ -1007,9 +1011,23 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.stats = static_cast<Q18Stats *>(e->arena.get("q18.stats", sizeof(Q18Stats)));
     s.stat_part = static_cast<Q18Stats *>(e->arena.get("q18.statpart", sizeof(Q18Stats) * 8 * e->num_sms));
     s.ticket = static_cast<unsigned int *>(e->arena.get("q18.ticket", 64, true, e->compute));
-    s.rows = static_cast<Q18Row *>(e->arena.get("q18.rows", sizeof(Q18Row) * std::max<uint64_t>(n_o, 1)));
-    s.amt = static_cast<long long *>(e->arena.get("q18.amt", 8 * std::max<uint64_t>(n_o, 1)));
+    s.rows = static_cast<Q18Row *>(e->arena.get("q18.rows", sizeof(Q18Row) * std::max<uint64_t>(rows_cap, 1)));
+    s.amt = static_cast<long long *>(e->arena.get("q18.amt", 8 * std::max<uint64_t>(rows_cap, 1)));
+    s.cand = nullptr;
+    s.ncand = nullptr;
     q.r->plan_flags = (s.jo.dense ? 1u : 0u) | (s.jc.dense ? 2u : 0u);
+}
+
+void q18_gather_and_order(h2tap_engine *e, QueryCtx &q, uint64_t n_rows_max);
+
+void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
+    const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
+    need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}, "Q18");
+    need_cols(v, O, {H2TAP_O_W_ID, H2TAP_O_D_ID, H2TAP_O_ID, H2TAP_O_C_ID, H2TAP_O_OL_CNT, H2TAP_O_ENTRY_D}, "Q18");
+    need_cols(v, C, {H2TAP_C_W_ID, H2TAP_C_D_ID, H2TAP_C_ID, H2TAP_C_LAST}, "Q18");
+    const uint64_t n_ol = v.n[OL], n_o = v.n[O], n_c = v.n[C];
+    q18_scratch(e, v, q, n_o);
+    Q18Scratch &s = q.q18;
 
     e->prof.run("q18_init", [&] { launch_q18_init(s, n_o, e->num_sms, e->compute); });
     e->prof.run("q18_build", [&] {
@@ -1032,9 +1050,16 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
                               n_o, colp<int32_t>(v, C, H2TAP_C_LAST), q.p[0], s, e->num_sms, e->compute);
     });
     CK(cudaGetLastError());
+    q18_gather_and_order(e, q, n_o);
+}
+
+// a7 + a8 of Q18 (and Q3): with world > 1 gather every rank's result rows to rank 0, then the
+// ORDER BY on the device and the scalar read-backs. `n_rows_max` bounds the local row count.
+void q18_gather_and_order(h2tap_engine *e, QueryCtx &q, uint64_t n_rows_max) {
+    Q18Scratch &s = q.q18;
     q.rows = s.rows;
     q.amt = s.amt;
-    q.n_max = n_o;
+    q.n_max = n_rows_max;
     Q18Small *sm = static_cast<Q18Small *>(q.small.first);
     if (e->world > 1) {
         // a7: groups are warehouse-local; gather the result rows to rank 0 (host-sized NCCL calls)
@@ -1048,7 +1073,7 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
         CK(cudaMemcpyAsync(&err_any, flag, 4, cudaMemcpyDeviceToHost, e->compute));
         sync_compute(e);
         if (sm->err) return;  // finish raises the local error
-        if (err_any) raise(H2TAP_EPLAN, "Q18: failed on another rank");
+        if (err_any) raise(H2TAP_EPLAN, "Q%u: failed on another rank", q.plan);
         auto *cnt_dev = static_cast<unsigned long long *>(e->arena.get("q18.allcnt", 8ull * e->world));
         NK(ncclAllGather(s.nout, cnt_dev, 1, ncclUint64, e->comm, e->compute));
         std::vector<unsigned long long> cnts(e->world);
@@ -1099,21 +1124,69 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     CK(cudaMemcpyAsync(&sm->tie, q.tie_dev, 4, cudaMemcpyDeviceToHost, e->compute));
 }
 
+// ---- NEXT-2: CH Q3 (customer ⋈ new_order ⋈ orders ⋈ order_line) on the Q18 machinery
+void launch_q3_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
+    const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER, NO = H2TAP_T_NEW_ORDER;
+    need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}, "Q3");
+    need_cols(v, O, {H2TAP_O_W_ID, H2TAP_O_D_ID, H2TAP_O_ID, H2TAP_O_C_ID, H2TAP_O_OL_CNT, H2TAP_O_ENTRY_D}, "Q3");
+    need_cols(v, C, {H2TAP_C_W_ID, H2TAP_C_D_ID, H2TAP_C_ID, H2TAP_C_STATE_P2}, "Q3");
+    need_cols(v, NO, {H2TAP_NO_W_ID, H2TAP_NO_D_ID, H2TAP_NO_O_ID}, "Q3");
+    const uint64_t n_ol = v.n[OL], n_o = v.n[O], n_c = v.n[C], n_no = v.n[NO];
+    const uint64_t cap = std::min<uint64_t>(n_o, n_no);  // result rows <= distinct marked orders
+    q18_scratch(e, v, q, cap);
+    Q18Scratch &s = q.q18;
+    s.cand = static_cast<unsigned int *>(e->arena.get("q3.cand", 4 * std::max<uint64_t>(cap, 1)));
+    s.ncand = static_cast<unsigned long long *>(e->arena.get("q3.ncand", 64));
+    e->prof.run("q3_init", [&] { launch_q18_init(s, n_o, e->num_sms, e->compute); });
+    e->prof.run("q3_build", [&] {
+        launch_q18_build(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
+                         colp<int32_t>(v, O, H2TAP_O_ID), n_o, colp<int32_t>(v, C, H2TAP_C_W_ID),
+                         colp<int32_t>(v, C, H2TAP_C_D_ID), colp<int32_t>(v, C, H2TAP_C_ID), n_c, s,
+                         e->num_sms, e->compute);
+    });
+    e->prof.run("q3_mark", [&] {
+        if (n_no)
+            launch_q3_mark(colp<int32_t>(v, NO, H2TAP_NO_W_ID), colp<int32_t>(v, NO, H2TAP_NO_D_ID),
+                           colp<int32_t>(v, NO, H2TAP_NO_O_ID), n_no, colp<int32_t>(v, O, H2TAP_O_W_ID),
+                           colp<int32_t>(v, O, H2TAP_O_D_ID), colp<int32_t>(v, O, H2TAP_O_C_ID),
+                           colp<int64_t>(v, O, H2TAP_O_ENTRY_D), colp<int32_t>(v, C, H2TAP_C_STATE_P2),
+                           q.p[0], (int)q.p[1], s, e->num_sms, e->compute);
+    });
+    e->prof.run("q3_probe_groupjoin", [&] {
+        if (n_ol && n_no)
+            launch_q3_probe(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
+                            colp<int32_t>(v, OL, H2TAP_OL_O_ID), colp<int64_t>(v, OL, H2TAP_OL_AMOUNT),
+                            n_ol, s, e->num_sms, e->compute);
+    });
+    e->prof.run("q3_emit", [&] {
+        if (cap)
+            launch_q3_emit(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
+                           colp<int32_t>(v, O, H2TAP_O_ID), colp<int32_t>(v, O, H2TAP_O_C_ID),
+                           colp<int32_t>(v, O, H2TAP_O_OL_CNT), colp<int64_t>(v, O, H2TAP_O_ENTRY_D), cap, s,
+                           e->num_sms, e->compute);
+    });
+    CK(cudaGetLastError());
+    q18_gather_and_order(e, q, cap);
+}
+
 void finish_q18(h2tap_engine *e, QueryCtx &q) {
     ResultImpl *r = q.r.get();
     Q18Small *sm = static_cast<Q18Small *>(q.small.first);
-    const char *names[] = {"c_last", "c_id", "o_id", "o_entry_d", "o_ol_cnt", "amount_sum", "o_w_id", "o_d_id"};
-    const uint32_t types[] = {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I32};
+    const bool q3 = q.plan == H2TAP_Q3;  // Q3 returns 5 of the sorted columns (R33)
+    const char *const *names = q3 ? kQ3Names : kQ18Names;
+    const uint32_t *types = q3 ? kQ3Types : kQ18Types;
+    const int ncols = q3 ? 5 : 8;
     if (q.q18_sorted_on_host_sync) {  // world > 1, rank != 0
         r->nrows = 0;
-        for (int i = 0; i < 8; ++i) add_col(r, names[i], types[i], result_block(r, 8));
+        for (int i = 0; i < ncols; ++i) add_col(r, names[i], types[i], result_block(r, 8));
         release_dev_blocks(e, q);
         return;
     }
     const unsigned int err = sm->err;
-    if (err & kErrDupOrders) raise(H2TAP_EDUPKEY, "Q18: duplicate orders primary key (w, d, o_id)");
-    if (err & kErrDupCustomer) raise(H2TAP_EDUPKEY, "Q18: duplicate customer primary key (w, d, c_id)");
-    if (err & kErrDomain) raise(H2TAP_EPLAN, "Q18: join key outside the supported domain");
+    const unsigned pl = q.plan;
+    if (err & kErrDupOrders) raise(H2TAP_EDUPKEY, "Q%u: duplicate orders primary key (w, d, o_id)", pl);
+    if (err & kErrDupCustomer) raise(H2TAP_EDUPKEY, "Q%u: duplicate customer primary key (w, d, c_id)", pl);
+    if (err & kErrDomain) raise(H2TAP_EPLAN, "Q%u: join key outside the supported domain", pl);
     const uint64_t nout = sm->nout;
     if (sm->tie && nout > 1) {
         // a run of > 32 equal 64-bit prefixes, or a bucket larger than shared memory: redo
@@ -1133,16 +1206,19 @@ void finish_q18(h2tap_engine *e, QueryCtx &q) {
         CK(cudaGetLastError());
     }
     r->nrows = nout;
-    const void *src[8] = {q.out.c_last, q.out.c_id, q.out.o_id, q.out.o_entry_d, q.out.o_ol_cnt,
-                          q.out.amount_sum, q.out.o_w_id, q.out.o_d_id};
-    const size_t es[8] = {4, 4, 4, 8, 4, 8, 4, 4};
+    const void *src18[8] = {q.out.c_last, q.out.c_id, q.out.o_id, q.out.o_entry_d, q.out.o_ol_cnt,
+                            q.out.amount_sum, q.out.o_w_id, q.out.o_d_id};
+    const void *src3[5] = {q.out.o_id, q.out.o_w_id, q.out.o_d_id, q.out.amount_sum, q.out.o_entry_d};
+    const void *const *src = q3 ? src3 : src18;
+    const size_t es18[8] = {4, 4, 4, 8, 4, 8, 4, 4}, es3[5] = {4, 4, 4, 8, 8};
+    const size_t *es = q3 ? es3 : es18;
     if (r->on_device) {
-        for (int i = 0; i < 8; ++i) add_col(r, names[i], types[i], src[i]);
+        for (int i = 0; i < ncols; ++i) add_col(r, names[i], types[i], src[i]);
         give_blocks_to_result(q);
         if (sm->tie) sync_compute(e);
         return;
     }
-    for (int i = 0; i < 8; ++i) {
+    for (int i = 0; i < ncols; ++i) {
         void *h = result_block(r, nout * es[i]);
         if (nout) CK(cudaMemcpyAsync(h, src[i], nout * es[i], cudaMemcpyDeviceToHost, e->compute));
         add_col(r, names[i], types[i], h);
@@ -1373,6 +1449,8 @@ constexpr int64_t kQ14Prefix = 0x5052;              // 'P' << 8 | 'R'  (LIKE 'PR
 constexpr int64_t kQ12DHi = 1577836800000000LL;     // 2020-01-01 00:00:00
 constexpr int64_t kQ4ELo = 1167696000000000LL;      // 2007-01-02 00:00:00
 constexpr int64_t kQ4EHi = 1325462400000000LL;      // 2012-01-02 00:00:00
+constexpr int64_t kQ3ELo = 1167696000000000LL;      // 2007-01-02 00:00:00
+constexpr int64_t kQ3Prefix = 0x4100;               // 'A' << 8  (LIKE 'A%')
 
 h2tap_status parse_query(const h2tap_query &in, QueryCtx &q) {
     uint32_t want;
@@ -1383,6 +1461,7 @@ h2tap_status parse_query(const h2tap_query &in, QueryCtx &q) {
         case H2TAP_Q14: want = 3; q.p[0] = kQ14DLo; q.p[1] = kQ14DHi; q.p[2] = kQ14Prefix; break;
         case H2TAP_Q12: want = 1; q.p[0] = kQ12DHi; break;
         case H2TAP_Q4: want = 2; q.p[0] = kQ4ELo; q.p[1] = kQ4EHi; break;
+        case H2TAP_Q3: want = 2; q.p[0] = kQ3ELo; q.p[1] = kQ3Prefix; break;
         default: return fail(H2TAP_EINVAL, "unknown plan id %u", in.plan_id);
     }
     if (in.nparams) {
@@ -1390,10 +1469,15 @@ h2tap_status parse_query(const h2tap_query &in, QueryCtx &q) {
             return fail(H2TAP_EINVAL, "plan %u takes %u params, got %u", in.plan_id, want, in.nparams);
         std::memcpy(q.p, in.params, sizeof(int64_t) * want);
     }
+    if (in.plan_id == H2TAP_Q3 && (q.p[1] < 0 || q.p[1] > 0xffff || ((q.p[1] & 0xff) && !(q.p[1] & 0xff00))))
+        return fail(H2TAP_EINVAL, "Q3: prefix must be (c0 << 8) | c1 with c0 != 0 when c1 != 0");
     q.plan = in.plan_id;
     q.flags = in.flags;
     return H2TAP_OK;
 }
+
+// Plans sharing scratch: Q3 runs on Q18's join scratch and ORDER BY buffers.
+uint32_t scratch_group(uint32_t plan) { return plan == H2TAP_Q3 ? (uint32_t)H2TAP_Q18 : plan; }
 
 h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2tap_result **out) {
     const auto t0 = std::chrono::steady_clock::now();
@@ -1442,7 +1526,7 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
             switch (q.plan) {
                 case H2TAP_Q1: finish_q1(e, q); break;
                 case H2TAP_Q6: finish_q6(e, q); break;
-                case H2TAP_Q18: finish_q18(e, q); break;
+                case H2TAP_Q18: case H2TAP_Q3: finish_q18(e, q); break;
                 case H2TAP_Q14: finish_q14(e, q); break;
                 case H2TAP_Q12: finish_groups(e, q, "Q12", "high_line_count", "low_line_count"); break;
                 case H2TAP_Q4: finish_groups(e, q, "Q4", "order_count", nullptr); break;
@@ -1452,7 +1536,7 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
     for (size_t i = 0; i < ctx.size(); ++i) {
         QueryCtx &q = ctx[i];
         for (size_t j = done; j < i; ++j)
-            if (ctx[j].plan == q.plan) { finish_upto(i); break; }
+            if (scratch_group(ctx[j].plan) == scratch_group(q.plan)) { finish_upto(i); break; }
         q.r.reset(new_result(e, *v, q.flags & H2TAP_RESULT_DEVICE));
         q.small = e->host_pool->get(256);
         if (!q.begin) {
@@ -1466,6 +1550,7 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
             case H2TAP_Q1: launch_q1_plan(e, *v, q); break;
             case H2TAP_Q6: launch_q6_plan(e, *v, q); break;
             case H2TAP_Q18: launch_q18_plan(e, *v, q); break;
+            case H2TAP_Q3: launch_q3_plan(e, *v, q); break;
             case H2TAP_Q14: launch_q14_plan(e, *v, q); break;
             case H2TAP_Q12: launch_q12_plan(e, *v, q); break;
             case H2TAP_Q4: launch_q4_plan(e, *v, q); break;
@@ -1578,7 +1663,7 @@ h2tap_status h2tap_load_snapshot_ex(h2tap_engine *e, const h2tap_table *tables, 
 
 h2tap_status h2tap_reserve(h2tap_engine *e, uint32_t table_id, uint64_t rows) {
     if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
-    if (table_id < 1 || table_id > 4) return fail(H2TAP_EINVAL, "unknown table id %u", table_id);
+    if (table_id < 1 || table_id >= (uint32_t)kTables) return fail(H2TAP_EINVAL, "unknown table id %u", table_id);
     return guarded([&]() -> h2tap_status {
         std::lock_guard<std::mutex> g(e->load_mu);
         CK(cudaSetDevice(e->device));

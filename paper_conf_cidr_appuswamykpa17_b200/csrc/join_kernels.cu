@@ -46,6 +46,7 @@ __global__ void q18_init_kernel(Q18Scratch s) {
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         *s.err = 0;
         *s.nout = 0;
+        if (s.ncand) *s.ncand = 0;
         Q18Stats st;
         st.amt_min = INT64_MAX; st.amt_max = INT64_MIN; st.ent_min = INT64_MAX; st.ent_max = INT64_MIN;
         st.w_min = INT32_MAX; st.w_max = INT32_MIN; st.d_min = INT32_MAX; st.d_max = INT32_MIN;
@@ -86,9 +87,18 @@ __device__ __forceinline__ bool eq3(const Key3 &a, const Key3 &b) {
     return (a.w == b.w) & (a.d == b.d) & (a.o == b.o);
 }
 
+// kFilter (CH Q3): only orders rows whose multiplier acc[row].pad is non-zero (set by the
+// new_order ⋈ orders ⋈ customer mark kernel) accumulate; the others skip their atomics.
+template <bool kFilter>
+__device__ __forceinline__ unsigned int keep_row(const Q18Scratch &s, unsigned int row) {
+    if (!kFilter || row == kNoRow) return row;
+    return __ldcg(&s.acc[row].pad) ? row : kNoRow;
+}
+
+template <bool kFilter>
 __device__ __forceinline__ void flush_run(const Q18Scratch &s, const Key3 &k, long long sum,
                                           unsigned int cnt) {
-    const unsigned int row = jx_lookup(s.jo, k.w, k.d, k.o);
+    const unsigned int row = keep_row<kFilter>(s, jx_lookup(s.jo, k.w, k.d, k.o));
     if (row != kNoRow) {
         atomicAdd(reinterpret_cast<unsigned long long *>(&s.acc[row].sum), (unsigned long long)sum);
         atomicAdd(&s.acc[row].cnt, cnt);
@@ -97,6 +107,7 @@ __device__ __forceinline__ void flush_run(const Q18Scratch &s, const Key3 &k, lo
 
 // One warp step over 128 consecutive rows, 4 per lane (k, a in registers; `valid` per lane):
 // in-lane runs, cross-lane segmented scan, one probe + two atomics per run (see above).
+template <bool kFilter>
 __device__ __forceinline__ void probe_lane_group(const Q18Scratch &s, const Key3 (&k)[4],
                                                  const long long (&a)[4], bool valid, int lane) {
         // in-lane runs: b[j] = row j starts a run; s[j], c[j] = running sum / count of its run
@@ -137,6 +148,10 @@ __device__ __forceinline__ void probe_lane_group(const Q18Scratch &s, const Key3
         unsigned int row[4];
 #pragma unroll
         for (int j = 0; j < 4; ++j) row[j] = f[j] ? jx_lookup(s.jo, k[j].w, k[j].d, k[j].o) : kNoRow;
+        if (kFilter) {
+#pragma unroll
+            for (int j = 0; j < 4; ++j) row[j] = keep_row<true>(s, row[j]);
+        }
 #pragma unroll
         for (int j = 0; j < 4; ++j)
             if (row[j] != kNoRow) {
@@ -145,6 +160,7 @@ __device__ __forceinline__ void probe_lane_group(const Q18Scratch &s, const Key3
             }
 }
 
+template <bool kFilter>
 __global__ void __launch_bounds__(kProbeThreads)
 q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ ol_d,
                  const int32_t *__restrict__ ol_o, const int64_t *__restrict__ ol_amt, uint64_t n,
@@ -182,12 +198,12 @@ q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ o
         } else {
             for (int j = 0; j < 4; ++j) { k[j] = {0, 0, 0}; a[j] = 0; }
         }
-        probe_lane_group(s, k, a, valid, lane);
+        probe_lane_group<kFilter>(s, k, a, valid, lane);
     }
     // ragged tail (< 4 rows) plus nothing else: one thread, row at a time
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         for (uint64_t i = nvec * 4; i < n; ++i)
-            flush_run(s, Key3{ol_w[i], ol_d[i], ol_o[i]}, ol_amt[i], 1u);
+            flush_run<kFilter>(s, Key3{ol_w[i], ol_d[i], ol_o[i]}, ol_amt[i], 1u);
     }
 }
 
@@ -263,10 +279,10 @@ q18_probe_tma_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict
         // rows of a partial last group (< 4, last chunk only) go one by one, straight from smem
         if (!valid && r < rows)
             for (unsigned j = r; j < rows; ++j)
-                flush_run(s, Key3{P.w[st][j], P.d[st][j], P.o[st][j]}, P.amt[st][j], 1u);
+                flush_run<false>(s, Key3{P.w[st][j], P.d[st][j], P.o[st][j]}, P.amt[st][j], 1u);
         __syncwarp();
         if (lane == 0) mbar_arrive(&P.empty[st]);  // registers hold everything from here on
-        probe_lane_group(s, k, a, valid, lane);
+        probe_lane_group<false>(s, k, a, valid, lane);
     }
 }
 
@@ -453,6 +469,109 @@ __global__ void q18_stats_kernel(const Q18Row *__restrict__ rows, const long lon
     stat.flush(part, ticket, st);
 }
 
+// ------------------------------------------------------------- CH Q3 (NEXT-2) --
+// Q3 = customer ⋈ new_order ⋈ orders ⋈ order_line, GROUP BY the orders key, ORDER BY revenue
+// DESC, o_entry_d. Its group key (ol_o_id, ol_w_id, ol_d_id, o_entry_d) is functionally
+// determined by the orders row (orders PK unique, checked), so the Q18 machinery applies:
+//  mark:  per new_order row, probe orders (o_entry_d > lo) then customer (c_state LIKE prefix);
+//         acc[orders row].pad counts the joined (new_order, customer) pairs — the inner join's
+//         multiplicity (a duplicated new_order row doubles the order's revenue); the first mark of
+//         a row appends it to a candidate list (count in *ncand, warp-aggregated);
+//  probe: q18_probe_kernel<true> (only marked rows accumulate);
+//  emit:  per candidate with >= 1 line, revenue = sum x multiplicity into 32-byte result rows +
+//         the sort-field statistics (row count in *nout), then the Q18 ORDER BY (same total
+//         order, R33).
+__device__ __forceinline__ bool like_prefix2(int p2, int prefix) {
+    // prefix = (c0 << 8) | c1 of a LIKE 'c0c1%' pattern; c1 == 0: one character; 0: empty pattern
+    const int mask = (prefix & 0xff) ? 0xffff : ((prefix & 0xff00) ? 0xff00 : 0);
+    return (p2 & mask) == prefix;
+}
+
+__global__ void q3_mark_kernel(const int32_t *__restrict__ no_w, const int32_t *__restrict__ no_d,
+                               const int32_t *__restrict__ no_o, uint64_t n_no,
+                               const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
+                               const int32_t *__restrict__ o_c, const int64_t *__restrict__ o_ent,
+                               const int32_t *__restrict__ c_p2, long long entry_lo, int prefix,
+                               Q18Scratch s) {
+    const int lane = threadIdx.x & 31;
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    const uint64_t n_pad = (n_no + 31) & ~31ull;  // whole warps iterate together (ballot below)
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n_pad; i += stride) {
+        unsigned int orow = kNoRow;
+        if (i < n_no) orow = jx_lookup(s.jo, __ldcs(no_w + i), __ldcs(no_d + i), __ldcs(no_o + i));
+        bool hit = false;
+        if (orow != kNoRow && __ldg(o_ent + orow) > entry_lo) {
+            const unsigned int crow = jx_lookup(s.jc, __ldg(o_w + orow), __ldg(o_d + orow), __ldg(o_c + orow));
+            hit = crow != kNoRow && like_prefix2(__ldg(c_p2 + crow), prefix);
+        }
+        bool first = false;
+        if (hit) first = atomicAdd(&s.acc[orow].pad, 1u) == 0u;
+        const unsigned int fb = __ballot_sync(kFull, first);
+        if (fb) {
+            unsigned long long base = 0;
+            if (lane == __ffs(fb) - 1) base = atomicAdd(s.ncand, (unsigned long long)__popc(fb));
+            base = __shfl_sync(kFull, base, __ffs(fb) - 1);
+            if (first) s.cand[base + __popc(fb & ((1u << lane) - 1))] = orow;
+        }
+    }
+}
+
+__global__ void __launch_bounds__(256)
+q3_emit_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
+               const int32_t *__restrict__ o_id, const int32_t *__restrict__ o_c,
+               const int32_t *__restrict__ o_cnt, const int64_t *__restrict__ o_ent, Q18Scratch s) {
+    __shared__ unsigned int wsum[8];
+    __shared__ unsigned long long s_base;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const uint64_t ncand = *s.ncand;  // written by the mark kernel (earlier on the stream)
+    StatAcc stat;
+    for (uint64_t base = (uint64_t)blockIdx.x * blockDim.x; base < ncand; base += (uint64_t)gridDim.x * blockDim.x) {
+        const uint64_t i = base + threadIdx.x;
+        unsigned int r = kNoRow;
+        long long sum = 0;
+        if (i < ncand) {
+            r = s.cand[i];
+            const ulonglong2 a = __ldcg(reinterpret_cast<const ulonglong2 *>(s.acc + r));
+            const unsigned int cnt = (unsigned int)a.y, mult = (unsigned int)(a.y >> 32);
+            if (cnt == 0) r = kNoRow;  // inner join: no order_line row, no group
+            sum = (long long)a.x * (long long)mult;
+        }
+        const unsigned int mine = r != kNoRow;
+        unsigned int x = mine;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const unsigned int t = __shfl_up_sync(kFull, x, o);
+            if (lane >= o) x += t;
+        }
+        if (lane == 31) wsum[warp] = x;
+        __syncthreads();
+        unsigned int before = 0, total = 0;
+#pragma unroll
+        for (int k = 0; k < 8; ++k) {
+            before += k < warp ? wsum[k] : 0u;
+            total += wsum[k];
+        }
+        if (threadIdx.x == 0) s_base = total ? atomicAdd(s.nout, (unsigned long long)total) : 0ull;
+        __syncthreads();
+        if (mine) {
+            const uint64_t p = s_base + before + x - 1;
+            Q18Row row;
+            row.o_entry_d = __ldg(o_ent + r);
+            row.c_last = 0;
+            row.c_id = __ldg(o_c + r);
+            row.o_id = __ldg(o_id + r);
+            row.o_ol_cnt = __ldg(o_cnt + r);
+            row.o_w_id = __ldg(o_w + r);
+            row.o_d_id = __ldg(o_d + r);
+            s.rows[p] = row;
+            s.amt[p] = sum;
+            stat.add(sum, row.o_entry_d, row.o_w_id, row.o_d_id, row.o_id);
+        }
+        __syncthreads();
+    }
+    stat.flush(s.stat_part, s.ticket, s.stats);
+}
+
 }  // namespace
 
 void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st) {
@@ -473,8 +592,33 @@ void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_i
 void launch_q18_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
                       const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
                       cudaStream_t st) {
-    q18_probe_kernel<<<grid_for((n_ol + 3) / 4, kProbeThreads, num_sms, 8), kProbeThreads, 0, st>>>(
+    q18_probe_kernel<false><<<grid_for((n_ol + 3) / 4, kProbeThreads, num_sms, 8), kProbeThreads, 0, st>>>(
         ol_w, ol_d, ol_o, ol_amt, n_ol, s);
+    count_launches(1);
+}
+
+void launch_q3_mark(const int32_t *no_w, const int32_t *no_d, const int32_t *no_o, uint64_t n_no,
+                    const int32_t *o_w, const int32_t *o_d, const int32_t *o_c, const int64_t *o_ent,
+                    const int32_t *c_p2, int64_t entry_lo, int prefix, const Q18Scratch &s, int num_sms,
+                    cudaStream_t st) {
+    q3_mark_kernel<<<grid_for(n_no, 256, num_sms, 8), 256, 0, st>>>(no_w, no_d, no_o, n_no, o_w, o_d, o_c,
+                                                                 o_ent, c_p2, entry_lo, prefix, s);
+    count_launches(1);
+}
+
+void launch_q3_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
+                     const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
+                     cudaStream_t st) {
+    q18_probe_kernel<true><<<grid_for((n_ol + 3) / 4, kProbeThreads, num_sms, 8), kProbeThreads, 0, st>>>(
+        ol_w, ol_d, ol_o, ol_amt, n_ol, s);
+    count_launches(1);
+}
+
+void launch_q3_emit(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, const int32_t *o_c,
+                    const int32_t *o_cnt, const int64_t *o_ent, uint64_t max_cand, const Q18Scratch &s,
+                    int num_sms, cudaStream_t st) {
+    // grid <= the stat_part capacity (8 blocks per SM); sized for the largest possible list
+    q3_emit_kernel<<<grid_for(max_cand, 256, num_sms, 8), 256, 0, st>>>(o_w, o_d, o_id, o_c, o_cnt, o_ent, s);
     count_launches(1);
 }
 

@@ -98,6 +98,9 @@ struct Q18Scratch {
     unsigned int *ticket;    // [1] last-block counter, zero-initialised once, self-resetting
     Q18Row *rows;            // [n_orders] unsorted result rows
     long long *amt;          // [n_orders] their amount_sum
+    // CH Q3 only (else null): orders rows marked by the new_order ⋈ customer step, and their count
+    unsigned int *cand;      // [n_new_order]
+    unsigned long long *ncand;// [1]
 };
 void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st);
 void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
@@ -113,6 +116,19 @@ void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_
                        const int32_t *o_c, const int32_t *o_cnt, const int64_t *o_ent,
                        uint64_t n_o, const int32_t *c_last, int64_t having,
                        const Q18Scratch &s, int num_sms, cudaStream_t st);
+// CH Q3 (NEXT-2) on the Q18 machinery: mark orders rows joined by new_order and an 'prefix%'
+// customer (multiplicity in acc[].pad, candidate list in cand / *ncand), probe order_line into the
+// marked rows only, emit result rows (revenue = sum x multiplicity, count *nout) + sort statistics.
+void launch_q3_mark(const int32_t *no_w, const int32_t *no_d, const int32_t *no_o, uint64_t n_no,
+                    const int32_t *o_w, const int32_t *o_d, const int32_t *o_c, const int64_t *o_ent,
+                    const int32_t *c_p2, int64_t entry_lo, int prefix, const Q18Scratch &s, int num_sms,
+                    cudaStream_t st);
+void launch_q3_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
+                     const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
+                     cudaStream_t st);
+void launch_q3_emit(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, const int32_t *o_c,
+                    const int32_t *o_cnt, const int64_t *o_ent, uint64_t max_cand, const Q18Scratch &s,
+                    int num_sms, cudaStream_t st);
 void launch_q18_stats(const Q18Row *rows, const long long *amt, uint64_t n, const Q18Scratch &s,
                       int num_sms, cudaStream_t st);  // recompute stats over gathered rows (multi-GPU)
 

@@ -1,5 +1,5 @@
 #!/usr/bin/env python
-"""NEXT-2 measurement: CH Q14 / Q12 / Q4 on one B200 at the bench workload (W=100, ~30 M
+"""NEXT-2 measurement: CH Q14 / Q12 / Q4 / Q3 on one B200 at the bench workload (W=100, ~30 M
 order_line rows, 'spread', seed 1), CH default parameters, snapshot resident in HBM.
 
 Per query: K timed runs (CUDA events on the engine stream around the query; L2 flushed between
@@ -10,6 +10,9 @@ Algorithmic bytes per kernel:
   q12_probe_groupby : 20 B x n_ol (w, d, o, delivery) + 20 B x n_o (slot 4, entry 8, carrier 4, cnt 4)
   q4_semijoin_mark  : 20 B x n_ol + 13 B x n_o (slot 4, entry 8, mark 1)
   q4_count          : 5 B x n_o (mark 1, o_ol_cnt 4)
+  q3_build          : 12 B x (n_o + n_c) read + 4 B x (n_o + n_c) slots + 16 B x n_o accumulators zeroed
+  q3_mark           : 12 B x n_no read + 4 B orders slot + 8 B o_entry_d per new_order row
+  q3_probe_groupjoin: 20 B x n_ol (w, d, o, amount) + 8 B x n_o (orders slot + multiplicity per run)
 Parity of the same queries at this size: tests/test_gpu_next2.py::test_full_size_w100.
 
 Usage: python scripts/ch_bench.py [--steps 20] [--warmup 3] [--out FILE]
@@ -36,19 +39,21 @@ def main():
     import torch
     import paper_conf_cidr_appuswamykpa17_b200 as h
     t = chgen.generate(1, a.warehouses + 1, seed=1)
-    plans_all = (h.H2TAP_Q14, h.H2TAP_Q12, h.H2TAP_Q4)
+    plans_all = (h.H2TAP_Q14, h.H2TAP_Q12, h.H2TAP_Q4, h.H2TAP_Q3)
     e = h.h2tap_open(0)
     h.h2tap_load_snapshot(e, h.hot_path_tables(t, plans_all), 1)
     n_ol, n_o = len(t["order_line"]["ol_o_id"]), len(t["orders"]["o_id"])
+    n_c, n_no = len(t["customer"]["c_id"]), len(t["new_order"]["no_o_id"])
     peak = json.load(open(os.path.join(ROOT, "MEASURED_PEAKS.json")))["hbm_gbs"] \
         if os.path.exists(os.path.join(ROOT, "MEASURED_PEAKS.json")) else 6650.0
     alg = {"q14_scan_join_sum": 20 * n_ol, "q12_build": 16 * n_o, "q4_build": 16 * n_o,
            "q12_probe_groupby": 20 * n_ol + 20 * n_o, "q4_semijoin_mark": 20 * n_ol + 13 * n_o,
-           "q4_count": 5 * n_o}
+           "q4_count": 5 * n_o, "q3_build": 16 * (n_o + n_c) + 16 * n_o, "q3_mark": 24 * n_no,
+           "q3_probe_groupjoin": 20 * n_ol + 8 * n_o}
     stream = torch.cuda.ExternalStream(h.h2tap_compute_stream(e))
     flush = torch.empty(512 << 20, dtype=torch.uint8, device="cuda")
     out = {}
-    for name, plan in (("q14", h.H2TAP_Q14), ("q12", h.H2TAP_Q12), ("q4", h.H2TAP_Q4)):
+    for name, plan in (("q14", h.H2TAP_Q14), ("q12", h.H2TAP_Q12), ("q4", h.H2TAP_Q4), ("q3", h.H2TAP_Q3)):
         ms = []
         for i in range(a.warmup + a.steps):
             flush.fill_(i & 0xff)
@@ -69,7 +74,7 @@ def main():
             r = h.h2tap_run_query(e, plan, None, flags=h.H2TAP_QUERY_PROFILE | h.H2TAP_RESULT_DEVICE)
             for k, v in r.kernels:
                 kern.setdefault(k, []).append(v)
-            flags = r.plan_flags
+            flags, nrows = r.plan_flags, r.nrows
             h.h2tap_free(r)
         kstats = {}
         for k, v in kern.items():
@@ -82,10 +87,11 @@ def main():
             kstats[k] = d
         out[name] = {"ms_median": round(float(np.median(ms)), 4), "ms_min": round(float(np.min(ms)), 4),
                      "order_line_rows_per_s": n_ol / (float(np.median(ms)) * 1e-3),
-                     "plan_flags": flags, "kernels": kstats}
+                     "plan_flags": flags, "result_rows": nrows, "kernels": kstats}
     h.h2tap_close(e)
-    line = json.dumps({"what": "NEXT-2 CH Q14/Q12/Q4, one B200, snapshot resident, L2 flushed per run",
+    line = json.dumps({"what": "NEXT-2 CH Q14/Q12/Q4/Q3, one B200, snapshot resident, L2 flushed per run",
                        "warehouses": a.warehouses, "order_line_rows": n_ol, "orders_rows": n_o,
+                       "customer_rows": n_c, "new_order_rows": n_no,
                        "peak_GBps": peak, "steps": a.steps, "queries": out})
     print(line)
     if a.out:
