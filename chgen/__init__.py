@@ -39,7 +39,7 @@ __all__ = [
     "DAY_US", "ts_us", "generate", "generate_item", "neworder_delta",
     "warehouse_ranges", "concat_tables", "TABLE_COLUMNS", "NewOrderState", "neworder_batch",
     "ROW_DTYPES", "to_records", "DeliveryState", "delivery_inputs", "delivery_batch",
-    "i_data_prefix2", "prefix2",
+    "i_data_prefix2", "prefix2", "layout_matrix", "encode_layout",
 ]
 
 
@@ -432,3 +432,32 @@ def delivery_batch(state: DeliveryState, w, carrier, clock0: int, step_us: int =
     return {"orders": {"o_carrier_id": (np.asarray(o_rows, np.uint32), np.asarray(o_vals, np.int32))},
             "order_line": {"ol_delivery_d": (np.asarray(l_rows, np.uint32),
                                              np.asarray(l_vals, np.int64))}}
+
+
+# ------------------------------------------------------- NEXT-3 layout table --
+def layout_matrix(nrows: int, ncols: int = 16, *, seed: int = 1, lo: int = -(1 << 20), hi: int = 1 << 20):
+    """The logical table of PAPER.md §5.3 (L965-972): ``nrows`` records of ``ncols`` int32
+    attributes, values uniform in [lo, hi) from stream Philox([seed, 2^43])."""
+    rng = np.random.Generator(np.random.Philox(key=np.array([seed, 1 << 43], dtype=np.uint64)))
+    return rng.integers(lo, hi, size=(nrows, ncols), dtype=np.int32)
+
+
+def encode_layout(m: np.ndarray, layout: str, *, pax_rows: int = 64, col_stride: int = 0) -> np.ndarray:
+    """Physical int32 array of logical matrix ``m`` (records x attributes) in ``layout``:
+    'nsm' = records back to back (row-major), 'dsm' = attributes back to back (column-major, column
+    starts ``col_stride`` elements apart, default nrows), 'pax' = pages of ncols minipages of
+    ``pax_rows`` values (the paper's 4 KB pages of 16 x 64; the last page zero-padded)."""
+    n, k = m.shape
+    if layout == "nsm":
+        return np.ascontiguousarray(m).reshape(-1)
+    if layout == "dsm":
+        stride = col_stride or n
+        out = np.zeros((k, stride), np.int32)
+        out[:, :n] = m.T
+        return out.reshape(-1)
+    if layout == "pax":
+        pages = -(-n // pax_rows)
+        pad = np.zeros((pages * pax_rows, k), np.int32)
+        pad[:n] = m
+        return np.ascontiguousarray(pad.reshape(pages, pax_rows, k).transpose(0, 2, 1)).reshape(-1)
+    raise ValueError(layout)

@@ -270,3 +270,22 @@ def q3(tables, entry_lo, prefix=b"A"):
         if n <= cap:
             return {k: v[:n] for k, v in out.items()}
         cap = n
+
+
+LAYOUTS = {"dsm": 1, "pax": 2, "nsm": 3}
+
+
+def layout_sum(data, layout, nrows, ncols, columns, *, col_stride=0, pax_rows=64):
+    """NEXT-3: SUM(col_c1 + ... + col_cN) over the physical int32 table ``data`` in ``layout``
+    ('dsm' / 'pax' / 'nsm'). Returns the sum, or None (NULL) for no rows."""
+    lib = _load()
+    lib.oracle_layout_sum.restype = C.c_int
+    a = np.ascontiguousarray(data, dtype=np.int32)
+    mask = 0
+    for c in columns:
+        mask |= 1 << int(c)
+    out, isnull = C.c_int64(), C.c_int32()
+    _check(lib.oracle_layout_sum(_p(a), C.c_int(LAYOUTS[layout]), C.c_int64(nrows), C.c_int64(ncols),
+                                 C.c_int64(col_stride or nrows), C.c_int64(pax_rows), C.c_uint64(mask),
+                                 C.byref(out), C.byref(isnull)))
+    return None if isnull.value else out.value

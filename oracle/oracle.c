@@ -530,3 +530,26 @@ done:
     map_free(&hc); map_free(&hn); map_free(&ho); map_free(&hg);
     return st == OR_OK ? ngroups : st;
 }
+
+/* ------------------------------------------------ layout scan (NEXT-3) -- */
+/* Address of record r, attribute c in each layout, as PAPER.md §5.3 describes them (L968-972). */
+static int64_t layout_addr(int layout, int64_t r, int64_t c, int64_t ncols, int64_t col_stride,
+                           int64_t pax_rows) {
+    if (layout == 1) return c * col_stride + r;                                       /* DSM */
+    if (layout == 2) return (r / pax_rows) * ncols * pax_rows + c * pax_rows + r % pax_rows;  /* PAX */
+    return r * ncols + c;                                                             /* NSM */
+}
+
+int oracle_layout_sum(const int32_t *data, int layout, int64_t nrows, int64_t ncols, int64_t col_stride,
+                      int64_t pax_rows, uint64_t col_mask, int64_t *sum, int32_t *is_null) {
+    int64_t total = 0;
+    for (int64_t r = 0; r < nrows; r++) {                 /* scan, one record at a time */
+        int64_t row = 0;                                   /* col_c1 + ... + col_cN */
+        for (int64_t c = 0; c < ncols; c++)
+            if (col_mask >> c & 1) row += data[layout_addr(layout, r, c, ncols, col_stride, pax_rows)];
+        if (__builtin_add_overflow(total, row, &total)) return OR_OVERFLOW;
+    }
+    *sum = total;
+    *is_null = nrows == 0;                                 /* SUM over no rows is NULL */
+    return OR_OK;
+}

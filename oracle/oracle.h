@@ -6,7 +6,7 @@
  * CUDA path (paper_conf_cidr_appuswamykpa17_b200/, include/), and never includes them.
  *
  * What it computes: the plain SQL definitions of CH-benCHmark Q1, Q6 and Q18, and (NEXT-2)
- * Q14, Q12, Q4 and Q3
+ * Q14, Q12, Q4 and Q3, and (NEXT-3) the paper's own layout query SUM(col1 + ... + colN)
  * (SURVEY.md Appendix A.1 [EXT]; the paper's OLAP path is PAPER.md L524-572, its only
  * query text is "TPC-H Q6, a selection over the lineitem table", L687-688), evaluated
  * row at a time, single-threaded, with SQL three-valued logic for NULLs.
@@ -129,6 +129,18 @@ int64_t oracle_q3(const or_customer *c, const or_new_order *no, const or_orders 
                   const or_order_line *ol, int64_t entry_lo, const char *prefix, int64_t cap,
                   int32_t *ol_o_id, int32_t *ol_w_id, int32_t *ol_d_id, int64_t *revenue,
                   int64_t *o_entry_d);
+
+/* NEXT-3 (§5.3): SELECT SUM(col_c1 + ... + col_cN) FROM dataset, for the
+ * attributes c with bit c of col_mask set, over a table of nrows records of ncols int32 attributes
+ * stored in one of the paper's three layouts (L968-972), value of record r, attribute c at:
+ *   layout 1 DSM (each attribute stored contiguously):  data[c * col_stride + r]
+ *   layout 2 PAX (pages of ncols minipages of pax_rows values; the paper: 16 x 64):
+ *            data[(r / pax_rows) * ncols * pax_rows + c * pax_rows + r % pax_rows]
+ *   layout 3 NSM (each record stored contiguously):      data[r * ncols + c]
+ * Per record the selected values are added in int64, then summed over records (overflow-checked).
+ * *is_null = 1 iff nrows == 0. Returns OR_OK or OR_OVERFLOW. */
+int oracle_layout_sum(const int32_t *data, int layout, int64_t nrows, int64_t ncols, int64_t col_stride,
+                      int64_t pax_rows, uint64_t col_mask, int64_t *sum, int32_t *is_null);
 
 #ifdef __cplusplus
 }
