@@ -37,7 +37,9 @@ H2TAP_T_ORDER_LINE, H2TAP_T_ORDERS, H2TAP_T_CUSTOMER, H2TAP_T_ITEM, H2TAP_T_NEW_
 H2TAP_Q1, H2TAP_Q6, H2TAP_Q18 = 1, 6, 18
 H2TAP_Q3, H2TAP_Q4, H2TAP_Q12, H2TAP_Q14 = 3, 4, 12, 14  # NEXT-2 CH queries
 H2TAP_FULL_RELOAD = 1
+H2TAP_DSM, H2TAP_PAX, H2TAP_NSM = 1, 2, 3  # NEXT-3 layouts (§5.3)
 H2TAP_LOAD_ASYNC = 1
+H2TAP_LOAD_ZERO_COPY = 2  # NEXT-4: kernels read the caller's pinned host columns over PCIe
 H2TAP_RESULT_DEVICE = 1
 H2TAP_QUERY_PROFILE = 2
 H2TAP_QUERY_HASH_JOIN = 4
@@ -114,7 +116,14 @@ class h2tap_result(C.Structure):
                 ("kernel_launches", C.c_uint64), ("plan_flags", C.c_uint32)]
 
 
+class h2tap_layout_table(C.Structure):
+    _fields_ = [("data", C.c_void_p), ("layout", C.c_uint32), ("ncols", C.c_uint32),
+                ("nrows", C.c_uint64), ("col_stride", C.c_uint64), ("pax_rows", C.c_uint32)]
+
+
 _P = C.c_void_p
+_lib.h2tap_layout_sum.argtypes = [_P, C.POINTER(h2tap_layout_table), C.c_uint64, C.POINTER(C.c_int64),
+                                  C.POINTER(C.c_int32), C.POINTER(C.c_double)]
 _lib.h2tap_open.argtypes = [C.POINTER(h2tap_config), C.POINTER(_P)]
 _lib.h2tap_load_snapshot_ex.argtypes = [_P, C.POINTER(h2tap_table), C.c_uint32, C.c_uint64, C.c_uint32]
 _lib.h2tap_load_snapshot.argtypes = [_P, C.POINTER(h2tap_table), C.c_uint32, C.c_uint64]
@@ -145,7 +154,7 @@ for _f in ("h2tap_open", "h2tap_load_snapshot_ex", "h2tap_load_snapshot", "h2tap
            "h2tap_reserve", "h2tap_refresh", "h2tap_refresh_rows", "h2tap_get_store_stats",
            "h2tap_sync",
            "h2tap_run_query_ex", "h2tap_run_query", "h2tap_run_queries", "h2tap_nccl_unique_id",
-           "h2tap_compute_stream"):
+           "h2tap_compute_stream", "h2tap_layout_sum"):
     getattr(_lib, _f).restype = C.c_int
 
 ABI_SYMBOLS = ["h2tap_open", "h2tap_load_snapshot", "h2tap_load_snapshot_ex",
@@ -153,7 +162,7 @@ ABI_SYMBOLS = ["h2tap_open", "h2tap_load_snapshot", "h2tap_load_snapshot_ex",
                "h2tap_get_store_stats", "h2tap_sync",
                "h2tap_run_query", "h2tap_run_query_ex", "h2tap_run_queries", "h2tap_free", "h2tap_close",
                "h2tap_last_error", "h2tap_nccl_unique_id", "h2tap_compute_stream",
-               "h2tap_c_last_name"]
+               "h2tap_c_last_name", "h2tap_layout_sum"]
 
 
 class H2tapError(RuntimeError):
@@ -507,3 +516,42 @@ def hot_path_tables(tables: dict, plans=HOT_PATH_PLANS) -> dict:
                 if c not in want[t]:
                     want[t].append(c)
     return {t: {c: tables[t][c] for c in cols} for t, cols in want.items()}
+
+
+def h2tap_layout_sum(engine: Engine, data, layout: int, nrows: int, ncols: int, columns, *,
+                     col_stride: int = 0, pax_rows: int = 64):
+    """NEXT-3 / NEXT-4: SELECT SUM(col_c1 + ... + col_cN) over an int32 table in ``layout``
+    (H2TAP_DSM / H2TAP_PAX / H2TAP_NSM, §5.3). ``data``: a CUDA int32 tensor (HBM) or a
+    PINNED CPU int32 tensor (read zero-copy over PCIe); ``columns``: attribute indices.
+    Returns (sum or None for no rows, kernel ms)."""
+    if not (hasattr(data, "data_ptr") and hasattr(data, "is_cuda")):
+        raise ValueError("data must be a torch tensor (CUDA, or pinned CPU)")
+    if data.is_cuda:  # the library's stream is not ordered after torch's: data must be written
+        import torch
+        torch.cuda.current_stream(data.device).synchronize()
+    mask = 0
+    for c in columns:
+        mask |= 1 << int(c)
+    t = h2tap_layout_table(data.data_ptr() if nrows else None, layout, ncols, nrows, col_stride, pax_rows)
+    out, isnull, ms = C.c_int64(), C.c_int32(), C.c_double()
+    _check(_lib.h2tap_layout_sum(engine.handle, C.byref(t), mask, C.byref(out), C.byref(isnull), C.byref(ms)))
+    return (None if isnull.value else out.value), ms.value
+
+
+def pinned_tables(tables: dict, capacity: dict | None = None, pad_rows: int = 64) -> dict:
+    """NEXT-4 helper: copy ``tables`` ({table: {column: array}}) into PINNED host torch tensors
+    for H2TAP_LOAD_ZERO_COPY. Each column's storage holds ``capacity[table]`` rows (default: its
+    length) plus ``pad_rows`` of readable slack; the returned tensors are views of the first n rows
+    — ``t.untyped_storage()`` spans the whole capacity, so later appends write rows in place and
+    publish them with ``first_row`` (see tests/test_gpu_zero_copy.py)."""
+    import torch
+    out = {}
+    for tname, cols in tables.items():
+        out[tname] = {}
+        for cname, a in cols.items():
+            arr = np.ascontiguousarray(a)
+            cap = max(len(arr), (capacity or {}).get(tname, 0))
+            buf = torch.empty(cap + pad_rows, dtype=getattr(torch, arr.dtype.name), pin_memory=True)
+            buf[:len(arr)].copy_(torch.from_numpy(arr))
+            out[tname][cname] = buf[:len(arr)]
+    return out

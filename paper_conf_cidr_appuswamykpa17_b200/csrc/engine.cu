@@ -207,6 +207,13 @@ struct View {  // immutable snapshot at one epoch (the paper's shallow-copied to
     // column statistics of the visible rows (zone map): valid once the view is published
     int smin[kTables][kStatCols], smax[kTables][kStatCols];
     bool has_stats[kTables] = {};
+    // NEXT-4: columns read zero-copy from the caller's pinned host memory (col[][] is then the
+    // mapped device address; nothing is kept alive by the view: the caller owns the memory)
+    bool host[kTables][kMaxCols] = {};
+    bool any_host(int t, std::initializer_list<int> cs) const {
+        for (int c : cs) if (host[t][c]) return true;
+        return false;
+    }
 };
 using ViewP = std::shared_ptr<const View>;
 
@@ -216,12 +223,14 @@ struct ColState {
     // bit is set in `bits` (copy-on-write of in-place updates, store_kernels.cu); bits_next is
     // the map the next update fills
     DevBufP cur, alt, bits, bits_next;
+    const char *host_base = nullptr;  // NEXT-4 zero-copy column: mapped address of row 0
     uint64_t cap_rows = 0;
     bool alt_valid = false;
     uint64_t alt_synced = 0;
 };
 struct TableState {
     bool present = false;
+    bool zero_copy = false; // NEXT-4: the table's columns live in the caller's pinned host memory
     uint32_t colmask = 0;   // which column ids this table carries (fixed at first load)
     uint64_t loaded = 0;    // rows copied or in flight
     ColState col[kMaxCols];
@@ -478,6 +487,28 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
             mask |= 1u << col.column_id;
         }
         const TableState &ts = e->tables[t.table_id];
+        const bool zc = flags & H2TAP_LOAD_ZERO_COPY;
+        if (!(t.flags & H2TAP_FULL_RELOAD) && ts.present && ts.zero_copy != zc)
+            return fail(H2TAP_ESHAPE, "table %u: switching between HBM and zero-copy needs a full reload", t.table_id);
+        if (zc) {
+            for (uint32_t c = 0; c < t.ncols; ++c) {
+                const h2tap_column &col = t.cols[c];
+                const size_t es = type_size(col.type);
+                const char *base = static_cast<const char *>(col.host_data) - t.first_row * es;
+                if (!col.host_data || (reinterpret_cast<uintptr_t>(base) & 15))
+                    return fail(H2TAP_EINVAL, "table %u column %u: zero-copy data must be 16-byte aligned", t.table_id, col.column_id);
+                cudaPointerAttributes a{};
+                if (cudaPointerGetAttributes(&a, base) != cudaSuccess || a.type != cudaMemoryTypeHost || !a.devicePointer) {
+                    cudaGetLastError();
+                    return fail(H2TAP_EINVAL, "table %u column %u: zero-copy data must be pinned, mapped host memory",
+                                t.table_id, col.column_id);
+                }
+                const ColState &cs = ts.col[col.column_id];
+                if (!(t.flags & H2TAP_FULL_RELOAD) && ts.present && cs.host_base != static_cast<const char *>(a.devicePointer))
+                    return fail(H2TAP_ESHAPE, "table %u column %u: a zero-copy append must extend the same host buffer",
+                                t.table_id, col.column_id);
+            }
+        }
         if (t.flags & H2TAP_FULL_RELOAD) {
             if (t.first_row != 0) return fail(H2TAP_EINVAL, "table %u: full reload must start at row 0", t.table_id);
         } else {
@@ -516,6 +547,8 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
             }
             if (!(mask & (1u << u.column_id)))
                 return fail(H2TAP_EPLAN, "update %u: table %u column %u was never loaded", i, u.table_id, u.column_id);
+            if ((seen[u.table_id] && (flags & H2TAP_LOAD_ZERO_COPY)) || (!seen[u.table_id] && e->tables[u.table_id].zero_copy))
+                return fail(H2TAP_EPLAN, "update %u: table %u is zero-copy (host-resident): update the host rows instead", i, u.table_id);
             uint32_t mx = 0;
             for (uint64_t k = 0; k < u.n; ++k) mx = std::max(mx, u.row_ids[k]);
             if (u.n && mx >= rows)
@@ -548,16 +581,33 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
             for (int c = 0; c < kNcols[t.table_id]; ++c)
                 if (!(mask & (1u << c))) {
                     v->col[t.table_id][c] = nullptr;
+                    v->host[t.table_id][c] = false;
                     v->keep[t.table_id][c].reset();
                     ts.col[c] = ColState{};
                 }
             ts.colmask = mask;
         }
+        const bool zc = flags & H2TAP_LOAD_ZERO_COPY;
+        ts.zero_copy = zc;
         for (uint32_t c = 0; c < t.ncols; ++c) {
             const h2tap_column &col = t.cols[c];
             ColState &cs = ts.col[col.column_id];
             const size_t es = type_size(col.type);
             const uint64_t need = t.row_count + kPadRows;
+            if (zc) {
+                // NEXT-4: publish the caller's pinned rows [0, row_count) as they are — no copy;
+                // kernels read them over PCIe through the mapped address
+                cudaPointerAttributes a{};
+                CK(cudaPointerGetAttributes(&a, static_cast<const char *>(col.host_data) - t.first_row * es));
+                cs = ColState{};
+                cs.host_base = static_cast<const char *>(a.devicePointer);
+                v->col[t.table_id][col.column_id] = const_cast<char *>(cs.host_base);
+                v->keep[t.table_id][col.column_id].reset();
+                v->host[t.table_id][col.column_id] = true;
+                continue;
+            }
+            v->host[t.table_id][col.column_id] = false;
+            cs.host_base = nullptr;
             if (full) {
                 // never overwrite a buffer a live view may read: reuse the spare only when no
                 // view references it any more, else allocate
@@ -785,7 +835,7 @@ void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.done_counter = static_cast<unsigned int *>(e->arena.get("q6.counter", 64, true, e->compute));
     s.out = static_cast<long long *>(e->arena.get("q6.out", 64));
     e->prof.run("q6_scan_filter_sum", [&] {
-        (e->scan_tma ? launch_q6_tma : launch_q6)(
+        (e->scan_tma && !v.any_host(T, {H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}) ? launch_q6_tma : launch_q6)(
             colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D), colp<int32_t>(v, T, H2TAP_OL_QUANTITY),
             colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T], q.p[0], q.p[1], q.p[2], q.p[3], s,
             e->num_sms, e->compute);
@@ -835,7 +885,7 @@ void launch_q1_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.o_cnt = static_cast<long long *>(dev_block(e, q, 8 * kQ1MaxGroups));
     if (fresh) launch_q1_reset(s, e->compute);  // tables self-clean afterwards (q1_compact)
     e->prof.run("q1_scan_filter_groupby", [&] {
-        (e->scan_tma ? launch_q1_tma : launch_q1)(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
+        (e->scan_tma && !v.any_host(T, {H2TAP_OL_NUMBER, H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}) ? launch_q1_tma : launch_q1)(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
                   colp<int32_t>(v, T, H2TAP_OL_QUANTITY), colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T],
                   q.p[0], s, e->num_sms, e->compute);
         CK(cudaGetLastError());
@@ -1015,6 +1065,8 @@ void q18_scratch(h2tap_engine *e, const View &v, QueryCtx &q, uint64_t rows_cap)
     s.amt = static_cast<long long *>(e->arena.get("q18.amt", 8 * std::max<uint64_t>(rows_cap, 1)));
     s.cand = nullptr;
     s.ncand = nullptr;
+    s.qbits = nullptr;
+    s.qwords = 0;
     q.r->plan_flags = (s.jo.dense ? 1u : 0u) | (s.jc.dense ? 2u : 0u);
 }
 
@@ -1038,7 +1090,7 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     });
     e->prof.run("q18_probe_groupjoin", [&] {
         if (n_ol)
-            (e->probe_tma ? launch_q18_probe_tma : launch_q18_probe)(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
+            (e->probe_tma && !v.any_host(OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}) ? launch_q18_probe_tma : launch_q18_probe)(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
                              colp<int32_t>(v, OL, H2TAP_OL_O_ID), colp<int64_t>(v, OL, H2TAP_OL_AMOUNT),
                              n_ol, s, e->num_sms, e->compute);
     });
@@ -1137,6 +1189,8 @@ void launch_q3_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     Q18Scratch &s = q.q18;
     s.cand = static_cast<unsigned int *>(e->arena.get("q3.cand", 4 * std::max<uint64_t>(cap, 1)));
     s.ncand = static_cast<unsigned long long *>(e->arena.get("q3.ncand", 64));
+    s.qwords = (n_o + 31) / 32;
+    s.qbits = static_cast<unsigned int *>(e->arena.get("q3.bits", 4 * std::max<uint64_t>(s.qwords, 1)));
     e->prof.run("q3_init", [&] { launch_q18_init(s, n_o, e->num_sms, e->compute); });
     e->prof.run("q3_build", [&] {
         launch_q18_build(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
@@ -1713,11 +1767,80 @@ h2tap_status h2tap_get_store_stats(h2tap_engine *e, h2tap_store_stats *out) {
     });
 }
 
+// ---- NEXT-3 / NEXT-4: SUM(col_1 + ... + col_N) over a DSM / PAX / NSM table (§5.3)
+namespace {
+int log2_exact(uint64_t x) {
+    if (!x || (x & (x - 1))) return -1;
+    return 63 - __builtin_clzll(x);
+}
+}  // namespace
+
+h2tap_status h2tap_layout_sum(h2tap_engine *e, const h2tap_layout_table *t, uint64_t col_mask,
+                              int64_t *sum, int32_t *is_null, double *device_ms) {
+    if (!e || !t || !sum || !is_null) return fail(H2TAP_EINVAL, "NULL argument");
+    if (t->layout < H2TAP_DSM || t->layout > H2TAP_NSM) return fail(H2TAP_EINVAL, "unknown layout %u", t->layout);
+    if (t->ncols < 1 || t->ncols > 64) return fail(H2TAP_EINVAL, "ncols must be in [1, 64]");
+    const uint64_t all = t->ncols == 64 ? ~0ull : ((1ull << t->ncols) - 1);
+    if (!col_mask || (col_mask & ~all)) return fail(H2TAP_EINVAL, "column mask selects no column or one >= ncols");
+    const int log_ncols = log2_exact(t->ncols), log_mp = log2_exact(t->pax_rows);
+    uint64_t stride = t->col_stride ? t->col_stride : t->nrows;
+    if (t->layout != H2TAP_DSM && (log_ncols < 2)) return fail(H2TAP_EINVAL, "PAX/NSM need ncols a power of two >= 4");
+    if (t->layout == H2TAP_PAX && log_mp < 2) return fail(H2TAP_EINVAL, "PAX needs pax_rows a power of two >= 4");
+    if (t->layout == H2TAP_DSM && stride < t->nrows) return fail(H2TAP_EINVAL, "DSM col_stride must be >= nrows");
+    if (t->layout == H2TAP_PAX && log_mp >= 2 &&
+        ((t->nrows + t->pax_rows - 1) >> log_mp) * (uint64_t)__builtin_popcountll(col_mask) >= (1ull << 32))
+        return fail(H2TAP_EINVAL, "PAX: pages x selected columns must be < 2^32");
+    if (t->nrows && (!t->data || (reinterpret_cast<uintptr_t>(t->data) & (t->layout == H2TAP_DSM ? 3 : 15))))
+        return fail(H2TAP_EINVAL, "data must be non-NULL and 16-byte aligned (4-byte for DSM)");
+    return guarded([&]() -> h2tap_status {
+        std::lock_guard<std::mutex> g(e->query_mu);
+        CK(cudaSetDevice(e->device));
+        const int32_t *dptr = static_cast<const int32_t *>(t->data);
+        if (t->nrows) {
+            // device memory, or pinned host memory reached through its mapped (UVA) address: the
+            // paper's zero-copy GPU access to host data (L568-572); pageable memory is refused
+            cudaPointerAttributes a{};
+            CK(cudaPointerGetAttributes(&a, t->data));
+            if (a.type == cudaMemoryTypeDevice || a.type == cudaMemoryTypeManaged) {
+                if (a.device != e->device) raise(H2TAP_EINVAL, "data lives on device %d, engine on %d", a.device, e->device);
+            } else if (a.type == cudaMemoryTypeHost) {
+                if (!a.devicePointer) raise(H2TAP_EINVAL, "pinned host data is not mapped into the device address space");
+                dptr = static_cast<const int32_t *>(a.devicePointer);
+            } else {
+                raise(H2TAP_EINVAL, "data is pageable host memory: pin it (cudaHostAlloc / cudaHostRegister)");
+            }
+        }
+        LayoutSel sel{};
+        for (int c = 0; c < 64; ++c)
+            if (col_mask >> c & 1) sel.col[sel.n++] = c;
+        auto *acc = static_cast<unsigned long long *>(e->arena.get("layout.acc", 64));
+        CK(cudaMemsetAsync(acc, 0, 8, e->compute));
+        CK(cudaEventRecord(e->q_begin, e->compute));
+        if (t->nrows)
+            launch_layout_sum(dptr, (int)t->layout, t->nrows, log_ncols, log_mp, stride, col_mask, sel, acc,
+                              e->num_sms, e->compute);
+        CK(cudaGetLastError());
+        CK(cudaEventRecord(e->q_end, e->compute));
+        unsigned long long host = 0;
+        CK(cudaMemcpyAsync(e->small_host, acc, 8, cudaMemcpyDeviceToHost, e->compute));
+        sync_compute(e);
+        std::memcpy(&host, e->small_host, 8);
+        float ms = 0;
+        CK(cudaEventElapsedTime(&ms, e->q_begin, e->q_end));
+        *sum = (int64_t)host;
+        *is_null = t->nrows == 0;  // SUM over no rows is NULL
+        if (device_ms) *device_ms = ms;
+        return H2TAP_OK;
+    });
+}
+
 h2tap_status h2tap_refresh_rows(h2tap_engine *e, const h2tap_row_table *tables, uint32_t ntables,
                                 const h2tap_update *updates, uint32_t nupdates, uint64_t epoch,
                                 uint32_t flags) {
     if (!e) return fail(H2TAP_EINVAL, "engine is NULL");
     if (ntables && !tables) return fail(H2TAP_EINVAL, "tables is NULL");
+    if (flags & H2TAP_LOAD_ZERO_COPY)
+        return fail(H2TAP_EINVAL, "zero-copy needs columns (DSM) in caller-owned pinned memory, not NSM records");
     return guarded([&]() -> h2tap_status {
         // column extraction NSM -> DSM into pinned buffers (the library's pinned block pool)
         std::vector<std::vector<h2tap_column>> cols(ntables);

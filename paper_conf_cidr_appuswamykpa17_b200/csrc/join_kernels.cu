@@ -36,12 +36,13 @@ unsigned grid_for(uint64_t work, int threads, int num_sms, int per_sm) {
 // Empties both join indexes, zeroes the group accumulators and the counters: one launch.
 // Empties both join indexes, zeroes the group accumulators and the counters: one launch.
 __global__ void q18_init_kernel(Q18Scratch s) {
-    const uint64_t a = jx_words(s.jo), b = jx_words(s.jc);
-    const uint64_t total = a + b;  // (the accumulators are zeroed by the build, row by row)
+    const uint64_t a = jx_words(s.jo), b = jx_words(s.jc), q = s.qbits ? s.qwords : 0;
+    const uint64_t total = a + b + q;  // (the accumulators are zeroed by the build, row by row)
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < total; i += stride) {
         if (i < a) jx_clear(s.jo, i);
-        else jx_clear(s.jc, i - a);
+        else if (i < a + b) jx_clear(s.jc, i - a);
+        else s.qbits[i - a - b] = 0u;
     }
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         *s.err = 0;
@@ -87,12 +88,13 @@ __device__ __forceinline__ bool eq3(const Key3 &a, const Key3 &b) {
     return (a.w == b.w) & (a.d == b.d) & (a.o == b.o);
 }
 
-// kFilter (CH Q3): only orders rows whose multiplier acc[row].pad is non-zero (set by the
-// new_order ⋈ orders ⋈ customer mark kernel) accumulate; the others skip their atomics.
+// kFilter (CH Q3): only orders rows marked by the new_order ⋈ orders ⋈ customer kernel
+// accumulate; the others skip their atomics.
+// The marks are read from a bitmap (n_orders / 8 bytes: L2-resident), not from acc[].pad.
 template <bool kFilter>
 __device__ __forceinline__ unsigned int keep_row(const Q18Scratch &s, unsigned int row) {
     if (!kFilter || row == kNoRow) return row;
-    return __ldcg(&s.acc[row].pad) ? row : kNoRow;
+    return (__ldcg(s.qbits + (row >> 5)) >> (row & 31)) & 1u ? row : kNoRow;
 }
 
 template <bool kFilter>
@@ -506,6 +508,7 @@ __global__ void q3_mark_kernel(const int32_t *__restrict__ no_w, const int32_t *
         }
         bool first = false;
         if (hit) first = atomicAdd(&s.acc[orow].pad, 1u) == 0u;
+        if (first) atomicOr(s.qbits + (orow >> 5), 1u << (orow & 31));
         const unsigned int fb = __ballot_sync(kFull, first);
         if (fb) {
             unsigned long long base = 0;

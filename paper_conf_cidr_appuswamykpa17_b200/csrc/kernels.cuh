@@ -101,6 +101,8 @@ struct Q18Scratch {
     // CH Q3 only (else null): orders rows marked by the new_order ⋈ customer step, and their count
     unsigned int *cand;      // [n_new_order]
     unsigned long long *ncand;// [1]
+    unsigned int *qbits;     // [qwords] bitmap of the marked orders rows (cleared by init)
+    unsigned long long qwords;
 };
 void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st);
 void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
@@ -266,5 +268,15 @@ void launch_q14(const int64_t *deliv, const int32_t *i_id, const int64_t *amt, u
                 int64_t d_hi, const ItemMap &m, const Q14Scratch &s, int num_sms, cudaStream_t st);
 void launch_q14_finalize(const Q14Scratch &s, cudaStream_t st);
 uint64_t launches_total();
+
+// ------------------------------ NEXT-3 / NEXT-4: layout scans (layout_kernels.cu) --
+// SUM(col_1 + ... + col_N) over int32 attributes in DSM / PAX / NSM (§5.3); `data` is a
+// device pointer or a mapped pinned host pointer (zero-copy over PCIe). *out accumulates (zero it).
+enum { kLayoutDsm = 1, kLayoutPax = 2, kLayoutNsm = 3 };
+constexpr int kMaxLayoutSel = 64;
+struct LayoutSel { int n; int col[kMaxLayoutSel]; };  // selected attribute indices
+void launch_layout_sum(const int32_t *data, int layout, uint64_t n, int log_ncols, int log_mp,
+                       uint64_t dsm_stride, unsigned long long mask, const LayoutSel &sel,
+                       unsigned long long *out, int num_sms, cudaStream_t st);
 
 }  // namespace h2tap

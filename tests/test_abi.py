@@ -38,7 +38,7 @@ def test_struct_layouts_match_header(h, tmp_path):
                "h2tap_config": h.h2tap_config, "h2tap_result": h.h2tap_result,
                "h2tap_field": h.h2tap_field, "h2tap_row_table": h.h2tap_row_table,
                "h2tap_query": h.h2tap_query, "h2tap_update": h.h2tap_update,
-               "h2tap_store_stats": h.h2tap_store_stats}
+               "h2tap_store_stats": h.h2tap_store_stats, "h2tap_layout_table": h.h2tap_layout_table}
     lines = ['#include <stdio.h>', '#include <stddef.h>', '#include "h2tap.h"', 'int main(void){']
     for name, cls in structs.items():
         lines.append(f'printf("{name} %zu\\n", sizeof({name}));')
