@@ -134,8 +134,11 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes):
         "q18_build": 12 * n_o + 12 * n_c + 16 * (n_o + n_c),
         "q18_probe_groupjoin": 20 * n_ol + 16 * n_o + 16 * n_o,
         "q18_having_compact": 16 * n_o + 28 * n_o + 16 * n_pass + 4 * n_pass + 40 * n_pass,
+        # ORDER BY v1 (H2TAP_ORDER=v1): (key, row id) sort, random row gather at emit
         "q18_sort_keys_hist": (32 + 8 + 8 + 4) * n_pass,   # rows + amounts -> keys + row ids
-        "q18_bucket_scatter": (12 + 12) * n_pass,          # read + write (key, row id)
+        # ORDER BY v2 (default): count matrix + scatter computing keys + chunked local sort
+        "q18_sort_hist": 8 * n_pass,                       # amounts (bucket bits inside field a)
+        "q18_bucket_scatter": (40 + 12) * n_pass if sort_passes == "v2" else (12 + 12) * n_pass,
         "q18_bucket_sort_emit": (12 + 32 + 40) * n_pass,   # (key, id), row gather, 8 result columns
     }.get(kernel)
 
@@ -297,7 +300,7 @@ def main():
 
     # ---- roofline for the dominant kernel (largest share of the step)
     kavg = {k: float(np.mean(v)) for k, v in kern.items()}
-    sort_passes = 0
+    sort_passes = "v1" if os.environ.get("H2TAP_ORDER") == "v1" else "v2"
     dominant = max(kavg, key=kavg.get) if kavg else None
     peak, peak_src = peaks()
     roof = None

@@ -308,6 +308,9 @@ struct h2tap_engine {
     // the Q18 probe keeps register prefetch at high occupancy — its dependent lookups and atomics
     // need more warps than a one-block-per-SM shared-memory ring leaves (H2TAP_PROBE=tma: ring)
     bool scan_tma = true, probe_tma = false;
+    // ORDER BY: payload-carrying bucket sort (v2); H2TAP_ORDER=v1 selects the (key, row id) sort
+    // with a random gather of the rows at emit (the A/B baseline)
+    bool order_v1 = false;
     // in-place updates copy only the dirty pages into the shadow (H2TAP_COW=full: always copy the
     // whole column — the A/B baseline of scripts/cow_bench.py)
     bool cow_full = false;
@@ -1042,8 +1045,14 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
             p.marks.push_back({name, {a, b}});
         }
     } marks(e->prof);
-    q18_bucket_order(q.rows, q.amt, q.plan_dev, n_max, bb, bs, d, q.tie_dev, e->num_sms, e->compute,
-                     &marks);
+    if (e->order_v1) {
+        q18_bucket_order(q.rows, q.amt, q.plan_dev, n_max, bb, bs, d, q.tie_dev, e->num_sms, e->compute,
+                         &marks);
+    } else {
+        bs.mat = static_cast<unsigned int *>(e->arena.get("q18.bmat", 4ull * ob_grid(e->num_sms) << kBucketMaxBits));
+        q18_bucket_order_v2(q.rows, q.amt, q.plan_dev, n_max, bb, bs, d, q.tie_dev, e->num_sms, e->compute,
+                            &marks);
+    }
 }
 
 // Scratch of the orders/customer group-join (Q18, and Q3 which reuses it): join indexes,
@@ -1687,6 +1696,7 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
                         prop.major, prop.minor);
         e->num_sms = prop.multiProcessorCount;
         if (const char *impl = std::getenv("H2TAP_SCAN")) e->scan_tma = std::strcmp(impl, "ldg") != 0;
+        if (const char *ob = std::getenv("H2TAP_ORDER")) e->order_v1 = std::strcmp(ob, "v1") == 0;
         if (const char *impl = std::getenv("H2TAP_PROBE")) e->probe_tma = std::strcmp(impl, "tma") == 0;
         if (const char *impl = std::getenv("H2TAP_COW")) e->cow_full = std::strcmp(impl, "full") == 0;
 

@@ -162,6 +162,7 @@ struct BucketSort {
     unsigned int *offset;  // [2^kBucketMaxBits + 1]
     unsigned int *big;     // [1 + 2^kBucketMaxBits]: count, then ids of buckets > small capacity
     unsigned int *ticket;  // [1], zero-initialised once, self-resetting
+    unsigned int *mat;     // v2: [ob_grid * 2^bucket_bits] per-partition bucket counts -> offsets
 };
 // Optional per-kernel profiling marks (the engine records CUDA events around each phase).
 struct PhaseMarks {
@@ -195,6 +196,12 @@ void launch_q18_plan(const Q18Stats *stats, const unsigned long long *nout, int 
 void q18_bucket_order(const Q18Row *rows, const long long *amt, const Q18Plan *plan, uint64_t n_max,
                       int bucket_bits, const BucketSort &s, const Q18Cols &dst, unsigned int *flag,
                       int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr);
+// Same contract, v2 (default): no global atomics in the partition (count matrix +
+// column scan), keys computed in the scatter; the per-bucket sort + emit kernels are v1's.
+int ob_grid(int num_sms);
+void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan *plan, uint64_t n_max,
+                         int bucket_bits, const BucketSort &s, const Q18Cols &dst, unsigned int *flag,
+                         int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr);
 // Within runs of equal prefix, order by the full tuple; runs longer than 32 raise *flag.
 // Exact fallback: three stable passes over the full fields (row rank, entry, amount).
 void launch_q18_field_keys(const Q18Row *rows, const long long *amt, const unsigned int *vals,

@@ -11,6 +11,7 @@
 //  * exact fallback (a run > 32 rows or a bucket > shared memory): one stable LSD radix sort of
 //    (key, row) pairs per field, r then e then a. Radix pass = per-tile digit histogram ->
 //    per-digit scan -> stable scatter; keys travel with their row ids.
+#include <algorithm>
 #include <cstdint>
 #include <cuda_runtime.h>
 
@@ -514,11 +515,22 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
             const unsigned int ns = 1u << sb, smask = ns - 1u;
             for (unsigned int i = threadIdx.x; i < ns; i += kBkThreads) S.sub[i] = 0;
             __syncthreads();
-            for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
-                const unsigned long long kk = k[lo + i];
-                S.k1[i] = kk;
-                S.v1[i] = v[lo + i];
-                atomicAdd(&S.sub[(unsigned int)(kk >> ssh) & smask], 1u);
+            for (unsigned int i0 = threadIdx.x; i0 < m; i0 += 2 * kBkThreads) {  // 2 loads in flight
+                unsigned long long kk[2];
+                unsigned int vv[2];
+#pragma unroll
+                for (int u = 0; u < 2; ++u) {
+                    const unsigned int i = i0 + u * kBkThreads;
+                    if (i < m) { kk[u] = __ldcs(k + lo + i); vv[u] = __ldcs(v + lo + i); }
+                }
+#pragma unroll
+                for (int u = 0; u < 2; ++u) {
+                    const unsigned int i = i0 + u * kBkThreads;
+                    if (i >= m) break;
+                    S.k1[i] = kk[u];
+                    S.v1[i] = vv[u];
+                    atomicAdd(&S.sub[(unsigned int)(kk[u] >> ssh) & smask], 1u);
+                }
             }
             __syncthreads();
             {   // exclusive scan of ns (<= 1024) sub-bucket counts: 4 per thread
@@ -593,27 +605,213 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
             }
         }
         __syncthreads();
-        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {  // emit at final positions
-            const unsigned int r = S.v1[i];
-            Q18Row row;
-            {
-                unsigned long long *w64 = reinterpret_cast<unsigned long long *>(&row);
-                ld16_policy(rows + r, w64[0], w64[1], drop);
-                ld16_policy(reinterpret_cast<const char *>(rows + r) + 16, w64[2], w64[3], drop);
+        for (unsigned int i0 = threadIdx.x; i0 < m; i0 += 2 * kBkThreads) {  // emit: 2 gathers in flight
+            Q18Row row[2];
+#pragma unroll
+            for (int u = 0; u < 2; ++u) {
+                const unsigned int i = i0 + u * kBkThreads;
+                if (i < m) {
+                    const unsigned int r = S.v1[i];
+                    unsigned long long *w64 = reinterpret_cast<unsigned long long *>(&row[u]);
+                    ld16_policy(rows + r, w64[0], w64[1], drop);
+                    ld16_policy(reinterpret_cast<const char *>(rows + r) + 16, w64[2], w64[3], drop);
+                }
             }
-            const unsigned long long a = sp.bits_a ? (S.k1[i] >> ashift) : 0ull;
-            const uint64_t j = lo + i;
-            dst.c_last[j] = row.c_last;
-            dst.c_id[j] = row.c_id;
-            dst.o_id[j] = row.o_id;
-            dst.o_entry_d[j] = row.o_entry_d;
-            dst.o_ol_cnt[j] = row.o_ol_cnt;
-            dst.amount_sum[j] = m == 1 && plan->n <= 1 ? amt[r]
-                                                       : (long long)((unsigned long long)sp.amt_max - a);
-            dst.o_w_id[j] = row.o_w_id;
-            dst.o_d_id[j] = row.o_d_id;
+#pragma unroll
+            for (int u = 0; u < 2; ++u) {
+                const unsigned int i = i0 + u * kBkThreads;
+                if (i >= m) break;
+                const unsigned long long a = sp.bits_a ? (S.k1[i] >> ashift) : 0ull;
+                const uint64_t j = lo + i;
+                dst.c_last[j] = row[u].c_last;
+                dst.c_id[j] = row[u].c_id;
+                dst.o_id[j] = row[u].o_id;
+                dst.o_entry_d[j] = row[u].o_entry_d;
+                dst.o_ol_cnt[j] = row[u].o_ol_cnt;
+                dst.amount_sum[j] = m == 1 && plan->n <= 1 ? amt[S.v1[i]]
+                                                           : (long long)((unsigned long long)sp.amt_max - a);
+                dst.o_w_id[j] = row[u].o_w_id;
+                dst.o_d_id[j] = row[u].o_d_id;
+            }
         }
         __syncthreads();
+    }
+}
+
+// ============================================== bucket sort v2 (default) ===
+// The v1 path above spends most of its time in global atomics (the histogram flush and the
+// per-block range reservation: ~one per row each) and in one shared-memory sort per ~360-row
+// bucket (eight block barriers per bucket, latency-bound). v2:
+//  1. ob_hist:    block b owns rows [b*T, (b+1)*T); shared histogram of the bucket ids (only
+//                 amount_sum is read when the bucket bits lie inside field a) -> matrix row b;
+//  2. ob_scan:    per bucket, exclusive scan down the [G][nb] matrix column (staged through
+//                 shared memory); the last block scans the bucket totals into bucket offsets;
+//  3. ob_scatter: block b seeds shared cursors with offset[j] + matrix[b][j] — no global atomics —
+//                 recomputes every key from the row and writes (key, row id) at its position;
+//  4. v1's per-bucket shared-memory sort + tie-fix + emit on the (key, row id) pairs.
+// Measured and rejected: carrying the 32-byte rows through the scatter (the
+// scattered 40 B/row writes cost more than the random gather they save) and sorting chunks of
+// whole buckets per block (fewer barriers, but 2 blocks/SM left the gathers latency-bound).
+constexpr int kObThreads = 1024;   // hist / scatter: 2 blocks of 32 warps per SM
+
+__device__ __forceinline__ unsigned int ob_bucket(const Q18Row *rows, const long long *amt, uint64_t i,
+                                                  const Q18SortSpec &sp, int shift, bool amt_only) {
+    if (amt_only) {  // the bucket bits are the top bits of field a
+        const unsigned long long a = field_a(amt[i], sp);
+        return (unsigned int)(a >> (shift - (sp.prefix_bits - sp.bits_a)));
+    }
+    return (unsigned int)(prefix_key(rows[i], amt[i], sp) >> shift);
+}
+
+__device__ __forceinline__ void ob_range(uint64_t n, uint64_t &r0, uint64_t &r1) {
+    const uint64_t T = (n + gridDim.x - 1) / gridDim.x;
+    r0 = (uint64_t)blockIdx.x * T;
+    r1 = r0 + T < n ? r0 + T : n;
+    if (r0 > n) r0 = n;
+}
+
+__global__ void __launch_bounds__(kObThreads)
+ob_hist_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
+               const Q18Plan *__restrict__ plan, int nb, unsigned int *__restrict__ mat) {
+    extern __shared__ unsigned int h[];
+    const uint64_t n = plan->n;
+    const Q18SortSpec sp = plan->spec;
+    const int shift = plan->shift;
+    const bool amt_only = sp.bits_a > 0 && shift >= sp.prefix_bits - sp.bits_a;
+    for (int i = threadIdx.x; i < nb; i += kObThreads) h[i] = 0;
+    __syncthreads();
+    uint64_t r0, r1;
+    ob_range(n, r0, r1);
+    constexpr int U = 8;
+    for (uint64_t i0 = r0 + threadIdx.x; i0 < r1; i0 += U * kObThreads) {
+        unsigned int b[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const uint64_t i = i0 + (uint64_t)u * kObThreads;
+            b[u] = i < r1 ? ob_bucket(rows, amt, i, sp, shift, amt_only) : 0xffffffffu;
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u)
+            if (b[u] != 0xffffffffu) atomicAdd(&h[b[u]], 1u);
+    }
+    __syncthreads();
+    unsigned int *row = mat + (uint64_t)blockIdx.x * nb;
+    for (int i = threadIdx.x; i < nb; i += kObThreads) row[i] = h[i];
+}
+
+// Column scans of the [G][nb] matrix: a block owns 32 buckets (lane); the [G][32] tile is staged
+// in shared memory with independent coalesced loads, scanned per column, written back. The last
+// block scans the bucket totals into bucket offsets.
+constexpr int kScanWarps = 8;
+__global__ void __launch_bounds__(32 * kScanWarps)
+ob_scan_kernel(unsigned int *__restrict__ mat, int G, int nb, unsigned int *__restrict__ count,
+               unsigned int *__restrict__ offset, unsigned int *ticket) {
+    extern __shared__ unsigned int tile[];  // [G][32]; the last block reuses it for nb totals
+    __shared__ bool last;
+    __shared__ unsigned int tot[kScanWarps][32];
+    __shared__ unsigned int wsum[kScanWarps];
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const int j = blockIdx.x * 32 + lane;
+#pragma unroll 8
+    for (int b = warp; b < G; b += kScanWarps) tile[b * 32 + lane] = j < nb ? __ldcs(mat + (uint64_t)b * nb + j) : 0u;
+    __syncthreads();
+    const int C = (G + kScanWarps - 1) / kScanWarps;
+    const int b0 = warp * C, b1 = min(G, b0 + C);
+    unsigned int sum = 0;
+    for (int b = b0; b < b1; ++b) sum += tile[b * 32 + lane];
+    tot[warp][lane] = sum;
+    __syncthreads();
+    unsigned int run = 0;
+    for (int w = 0; w < warp; ++w) run += tot[w][lane];
+    if (warp == kScanWarps - 1 && j < nb) count[j] = run + sum;
+    for (int b = b0; b < b1; ++b) {
+        const unsigned int c = tile[b * 32 + lane];
+        tile[b * 32 + lane] = run;
+        run += c;
+    }
+    __syncthreads();
+    if (j < nb) {
+#pragma unroll 8
+        for (int b = warp; b < G; b += kScanWarps) mat[(uint64_t)b * nb + j] = tile[b * 32 + lane];
+    }
+    __threadfence();
+    __syncthreads();
+    if (threadIdx.x == 0) last = atomicAdd(ticket, 1u) == gridDim.x - 1;
+    __syncthreads();
+    if (!last) return;
+    __threadfence();
+    // last block: stage the bucket totals in shared memory (all loads independent, many in
+    // flight), then an exclusive scan, warp-cooperatively (lane i reads element base + i: no bank
+    // conflicts), each warp over a contiguous range
+    unsigned int *sc = tile;  // reuse: nb entries (dynamic smem >= 4 * nb)
+#pragma unroll 8
+    for (int i = threadIdx.x; i < nb; i += 32 * kScanWarps) sc[i] = __ldcg(count + i);
+    __syncthreads();
+    const int span = (nb + kScanWarps - 1) / kScanWarps;
+    const int w0 = warp * span, w1 = min(nb, w0 + span);
+    unsigned int wtot = 0;
+    for (int base = w0; base < w1; base += 32) {
+        const int i = base + lane;
+        wtot += __reduce_add_sync(kFull, i < w1 ? sc[i] : 0u);
+    }
+    if (lane == 0) wsum[warp] = wtot;
+    __syncthreads();
+    unsigned int acc = 0;
+    for (int w = 0; w < warp; ++w) acc += wsum[w];
+    for (int base = w0; base < w1; base += 32) {
+        const int i = base + lane;
+        const unsigned int c = i < w1 ? sc[i] : 0u;
+        unsigned int x = c;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const unsigned int y = __shfl_up_sync(kFull, x, o);
+            if (lane >= o) x += y;
+        }
+        if (i < w1) offset[i] = acc + x - c;
+        acc += __shfl_sync(kFull, x, 31);
+    }
+    if (warp == kScanWarps - 1 && lane == 0) offset[nb] = acc;
+    if (threadIdx.x == 0) *ticket = 0;  // self-reset
+}
+
+__global__ void __launch_bounds__(kObThreads)
+ob_scatter_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
+                  const Q18Plan *__restrict__ plan, int nb, const unsigned int *__restrict__ mat,
+                  const unsigned int *__restrict__ offset, unsigned long long *__restrict__ kout,
+                  unsigned int *__restrict__ vout) {
+    extern __shared__ unsigned int cur[];
+    const uint64_t n = plan->n;
+    const Q18SortSpec sp = plan->spec;
+    const int shift = plan->shift;
+    const unsigned int *row = mat + (uint64_t)blockIdx.x * nb;
+    for (int i = threadIdx.x; i < nb; i += kObThreads) cur[i] = offset[i] + row[i];
+    __syncthreads();
+    uint64_t r0, r1;
+    ob_range(n, r0, r1);
+    constexpr int U = 4;
+    for (uint64_t i0 = r0 + threadIdx.x; i0 < r1; i0 += U * kObThreads) {
+        Q18Row r[U];
+        long long a[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const uint64_t i = i0 + (uint64_t)u * kObThreads;
+            if (i < r1) {
+                const ulonglong2 *src = reinterpret_cast<const ulonglong2 *>(rows + i);
+                ulonglong2 *d = reinterpret_cast<ulonglong2 *>(&r[u]);
+                d[0] = src[0];  // (rows stay cached: the emit gathers them again)
+                d[1] = src[1];
+                a[u] = __ldcs(amt + i);
+            }
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const uint64_t i = i0 + (uint64_t)u * kObThreads;
+            if (i >= r1) break;
+            const unsigned long long kk = prefix_key(r[u], a[u], sp);
+            const unsigned int p = atomicAdd(&cur[(unsigned int)(kk >> shift)], 1u);
+            kout[p] = kk;
+            vout[p] = (unsigned int)i;
+        }
     }
 }
 
@@ -666,6 +864,62 @@ void q18_bucket_order(const Q18Row *rows, const long long *amt, const Q18Plan *p
     bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall><<<(unsigned)num_sms, kBkThreads,
                                                           sizeof(LsSmem<kLsCapLarge>), st>>>(
         s.k[1], s.v[1], s.offset, nb, plan, rows, amt, dst, flag, s.big);
+    count_launches(1);
+    end();
+}
+
+}  // namespace h2tap
+
+namespace h2tap {
+
+int ob_grid(int num_sms) { return 2 * num_sms; }  // row partitions of the v2 ORDER BY front
+
+void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan *plan, uint64_t n_max,
+                         int bucket_bits, const BucketSort &s, const Q18Cols &dst, unsigned int *flag,
+                         int num_sms, cudaStream_t st, PhaseMarks *marks) {
+    auto begin = [&](const char *nm) { if (marks) marks->begin(nm); };
+    auto end = [&] { if (marks) marks->end(); };
+    if (bucket_bits > kBucketMaxBits) bucket_bits = kBucketMaxBits;
+    const int nb = 1 << bucket_bits;
+    const int G = ob_grid(num_sms);
+    static bool init = false;
+    if (!init) {
+        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapSmall, 0>,
+                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapSmall>));
+        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall>,
+                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapLarge>));
+        cudaFuncSetAttribute(ob_hist_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 << kBucketMaxBits);
+        cudaFuncSetAttribute(ob_scatter_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 << kBucketMaxBits);
+        cudaFuncSetAttribute(ob_scan_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             4 * std::max(32 * G, 1 << kBucketMaxBits));
+        init = true;
+    }
+    (void)n_max;
+    cudaMemsetAsync(s.big, 0, sizeof(unsigned int), st);
+    begin("q18_sort_hist");
+    ob_hist_kernel<<<G, kObThreads, nb * 4, st>>>(rows, amt, plan, nb, s.mat);
+    count_launches(1);
+    end();
+    begin("q18_sort_scan");
+    ob_scan_kernel<<<(nb + 31) / 32, 32 * kScanWarps, 4 * std::max(32 * G, nb), st>>>(s.mat, G, nb, s.count,
+                                                                                   s.offset, s.ticket);
+    count_launches(1);
+    end();
+    begin("q18_bucket_scatter");
+    ob_scatter_kernel<<<G, kObThreads, nb * 4, st>>>(rows, amt, plan, nb, s.mat, s.offset, s.k[0], s.v[0]);
+    count_launches(1);
+    end();
+    // per-bucket shared-memory sort + tie-fix + emit: the v1 kernels on the (key, row id) pairs
+    begin("q18_bucket_sort_emit");
+    const unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
+    bucket_local_emit_kernel<kLsCapSmall, 0><<<lb, kBkThreads, sizeof(LsSmem<kLsCapSmall>), st>>>(
+        s.k[0], s.v[0], s.offset, nb, plan, rows, amt, dst, flag, s.big);
+    count_launches(1);
+    end();
+    begin("q18_bucket_sort_emit_large");
+    bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall><<<(unsigned)num_sms, kBkThreads,
+                                                          sizeof(LsSmem<kLsCapLarge>), st>>>(
+        s.k[0], s.v[0], s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
     end();
 }

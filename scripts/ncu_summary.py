@@ -64,6 +64,9 @@ if traffic:
              "q18_keys_hist_kernel": "q18_sort_keys_hist", "bucket_scatter_kernel": "q18_bucket_scatter",
              "bucket_local_emit_kernel<2048, 0>": "q18_bucket_sort_emit",
              "bucket_local_emit_kernel<8192, 2048>": "q18_bucket_sort_emit_large",
+             "ob_hist_kernel": "q18_sort_hist", "ob_scan_kernel": "q18_sort_scan",
+             "ob_scatter_kernel": "q18_bucket_scatter", "ob_local_emit_kernel<2048, 0>": "q18_bucket_sort_emit",
+             "ob_local_emit_kernel<8192, 2048>": "q18_bucket_sort_emit_large",
              "q18_plan_kernel": "q18_plan", "q1_compact_kernel": "q1_compact",
              "q1_emit_kernel": "q1_emit"}
     bymark = {}
