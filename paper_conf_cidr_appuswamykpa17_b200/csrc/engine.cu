@@ -1001,6 +1001,9 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     const uint64_t n_max = std::max<uint64_t>(q.n_max, 1);
     int bb = 1;
     while (bb < kBucketMaxBits && (n_max >> (bb + 9)) > 0) ++bb;   // ~256-512 rows per bucket
+    if (!e->order_v1) bb = ob_bucket_bits(n_max);
+    if (const char *d = std::getenv("H2TAP_BUCKET_BITS_DELTA"))      // tuning knob
+        bb = std::max(1, std::min(kBucketMaxBits, bb + std::atoi(d)));
     q.plan_dev = static_cast<Q18Plan *>(e->arena.get("q18.plan", sizeof(Q18Plan)));
     e->prof.run("q18_plan", [&] { launch_q18_plan(q.q18.stats, q.q18.nout, bb, q.plan_dev, e->compute); });
     for (int b = 0; b < 2; ++b) {

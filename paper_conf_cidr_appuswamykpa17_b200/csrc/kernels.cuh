@@ -199,6 +199,7 @@ void q18_bucket_order(const Q18Row *rows, const long long *amt, const Q18Plan *p
 // Same contract, v2 (default): no global atomics in the partition (count matrix +
 // column scan), keys computed in the scatter; the per-bucket sort + emit kernels are v1's.
 int ob_grid(int num_sms);
+int ob_bucket_bits(uint64_t n_max);
 void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan *plan, uint64_t n_max,
                          int bucket_bits, const BucketSort &s, const Q18Cols &dst, unsigned int *flag,
                          int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr);

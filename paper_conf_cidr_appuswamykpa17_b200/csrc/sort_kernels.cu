@@ -653,6 +653,8 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
 // scattered 40 B/row writes cost more than the random gather they save) and sorting chunks of
 // whole buckets per block (fewer barriers, but 2 blocks/SM left the gathers latency-bound).
 constexpr int kObThreads = 1024;   // hist / scatter: 2 blocks of 32 warps per SM
+constexpr int kObCap = kLsCapSmall;  // per-bucket sort capacity: 2 048 rows (56 KB, 3 blocks/SM);
+                                     // 4 096 (2 blocks/SM) with ~730-row buckets measured slower
 
 __device__ __forceinline__ unsigned int ob_bucket(const Q18Row *rows, const long long *amt, uint64_t i,
                                                   const Q18SortSpec &sp, int shift, bool amt_only) {
@@ -873,6 +875,11 @@ void q18_bucket_order(const Q18Row *rows, const long long *amt, const Q18Plan *p
 namespace h2tap {
 
 int ob_grid(int num_sms) { return 2 * num_sms; }  // row partitions of the v2 ORDER BY front
+int ob_bucket_bits(uint64_t n_max) {  // ~256-512 rows per bucket
+    int bb = 1;
+    while (bb < kBucketMaxBits && (n_max >> (bb + 9)) > 0) ++bb;
+    return bb;
+}
 
 void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan *plan, uint64_t n_max,
                          int bucket_bits, const BucketSort &s, const Q18Cols &dst, unsigned int *flag,
@@ -884,9 +891,9 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
     const int G = ob_grid(num_sms);
     static bool init = false;
     if (!init) {
-        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapSmall, 0>,
-                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapSmall>));
-        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall>,
+        cudaFuncSetAttribute(bucket_local_emit_kernel<kObCap, 0>,
+                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kObCap>));
+        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapLarge, kObCap>,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapLarge>));
         cudaFuncSetAttribute(ob_hist_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 << kBucketMaxBits);
         cudaFuncSetAttribute(ob_scatter_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 << kBucketMaxBits);
@@ -912,12 +919,12 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
     // per-bucket shared-memory sort + tie-fix + emit: the v1 kernels on the (key, row id) pairs
     begin("q18_bucket_sort_emit");
     const unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
-    bucket_local_emit_kernel<kLsCapSmall, 0><<<lb, kBkThreads, sizeof(LsSmem<kLsCapSmall>), st>>>(
+    bucket_local_emit_kernel<kObCap, 0><<<lb, kBkThreads, sizeof(LsSmem<kObCap>), st>>>(
         s.k[0], s.v[0], s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
     end();
     begin("q18_bucket_sort_emit_large");
-    bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall><<<(unsigned)num_sms, kBkThreads,
+    bucket_local_emit_kernel<kLsCapLarge, kObCap><<<(unsigned)num_sms, kBkThreads,
                                                           sizeof(LsSmem<kLsCapLarge>), st>>>(
         s.k[0], s.v[0], s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
