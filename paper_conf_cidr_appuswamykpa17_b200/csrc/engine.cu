@@ -311,6 +311,11 @@ struct h2tap_engine {
     // ORDER BY: payload-carrying bucket sort (v2); H2TAP_ORDER=v1 selects the (key, row id) sort
     // with a random gather of the rows at emit (the A/B baseline)
     bool order_v1 = false;
+    // zero-copy (host-resident) columns are streamed by the TMA-bulk kernels (cp.async.bulk reads
+    // the mapped host memory: 0.92 of the PCIe copy rate vs 0.51 with LDG loads);
+    // H2TAP_ZC_TMA=0 selects the LDG kernels
+    bool zc_tma = true;
+    int having_unroll = 2;  // H2TAP_HAVING_UNROLL (2 or 4): orders rows per thread in the HAVING pass
     // in-place updates copy only the dirty pages into the shadow (H2TAP_COW=full: always copy the
     // whole column — the A/B baseline of scripts/cow_bench.py)
     bool cow_full = false;
@@ -838,7 +843,7 @@ void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.done_counter = static_cast<unsigned int *>(e->arena.get("q6.counter", 64, true, e->compute));
     s.out = static_cast<long long *>(e->arena.get("q6.out", 64));
     e->prof.run("q6_scan_filter_sum", [&] {
-        (e->scan_tma && !v.any_host(T, {H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}) ? launch_q6_tma : launch_q6)(
+        (e->scan_tma && (e->zc_tma || !v.any_host(T, {H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT})) ? launch_q6_tma : launch_q6)(
             colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D), colp<int32_t>(v, T, H2TAP_OL_QUANTITY),
             colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T], q.p[0], q.p[1], q.p[2], q.p[3], s,
             e->num_sms, e->compute);
@@ -888,7 +893,7 @@ void launch_q1_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.o_cnt = static_cast<long long *>(dev_block(e, q, 8 * kQ1MaxGroups));
     if (fresh) launch_q1_reset(s, e->compute);  // tables self-clean afterwards (q1_compact)
     e->prof.run("q1_scan_filter_groupby", [&] {
-        (e->scan_tma && !v.any_host(T, {H2TAP_OL_NUMBER, H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}) ? launch_q1_tma : launch_q1)(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
+        (e->scan_tma && (e->zc_tma || !v.any_host(T, {H2TAP_OL_NUMBER, H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT})) ? launch_q1_tma : launch_q1)(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
                   colp<int32_t>(v, T, H2TAP_OL_QUANTITY), colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T],
                   q.p[0], s, e->num_sms, e->compute);
         CK(cudaGetLastError());
@@ -1102,7 +1107,8 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     });
     e->prof.run("q18_probe_groupjoin", [&] {
         if (n_ol)
-            (e->probe_tma && !v.any_host(OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}) ? launch_q18_probe_tma : launch_q18_probe)(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
+            ((e->probe_tma || e->zc_tma) && (e->probe_tma || v.any_host(OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}))
+                 ? launch_q18_probe_tma : launch_q18_probe)(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
                              colp<int32_t>(v, OL, H2TAP_OL_O_ID), colp<int64_t>(v, OL, H2TAP_OL_AMOUNT),
                              n_ol, s, e->num_sms, e->compute);
     });
@@ -1111,7 +1117,8 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
             launch_q18_having(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
                               colp<int32_t>(v, O, H2TAP_O_ID), colp<int32_t>(v, O, H2TAP_O_C_ID),
                               colp<int32_t>(v, O, H2TAP_O_OL_CNT), colp<int64_t>(v, O, H2TAP_O_ENTRY_D),
-                              n_o, colp<int32_t>(v, C, H2TAP_C_LAST), q.p[0], s, e->num_sms, e->compute);
+                              n_o, colp<int32_t>(v, C, H2TAP_C_LAST), q.p[0], s, e->num_sms, e->compute,
+                              e->having_unroll);
     });
     CK(cudaGetLastError());
     q18_gather_and_order(e, q, n_o);
@@ -1700,6 +1707,8 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         e->num_sms = prop.multiProcessorCount;
         if (const char *impl = std::getenv("H2TAP_SCAN")) e->scan_tma = std::strcmp(impl, "ldg") != 0;
         if (const char *ob = std::getenv("H2TAP_ORDER")) e->order_v1 = std::strcmp(ob, "v1") == 0;
+        if (const char *z = std::getenv("H2TAP_ZC_TMA")) e->zc_tma = std::atoi(z) != 0;
+        if (const char *hu = std::getenv("H2TAP_HAVING_UNROLL")) e->having_unroll = std::atoi(hu) == 4 ? 4 : 2;
         if (const char *impl = std::getenv("H2TAP_PROBE")) e->probe_tma = std::strcmp(impl, "tma") == 0;
         if (const char *impl = std::getenv("H2TAP_COW")) e->cow_full = std::strcmp(impl, "full") == 0;
 

@@ -372,9 +372,7 @@ struct StatAcc {
 // Each block iteration covers kHavingRows consecutive orders rows (kHavingUnroll per thread);
 // passing rows get output slots from ONE atomicAdd per block iteration (block-wide exclusive
 // scan of the per-thread counts), so the output counter sees ~n/1024 atomics, not n/32.
-constexpr int kHavingUnroll = 2;
-constexpr int kHavingRows = kHavingThreads * kHavingUnroll;
-
+template <int kHavingUnroll>
 __global__ void __launch_bounds__(kHavingThreads, 4)
 q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
                   const int32_t *__restrict__ o_id, const int32_t *__restrict__ o_c,
@@ -383,6 +381,7 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
     __shared__ unsigned int wsum[kHavingThreads / 32];
     __shared__ unsigned long long s_base;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    constexpr int kHavingRows = kHavingThreads * kHavingUnroll;
     const uint64_t keep = l2_policy_evict_last();
     StatAcc stat;
     for (uint64_t base = (uint64_t)blockIdx.x * kHavingRows; base < n;
@@ -644,10 +643,13 @@ void launch_q18_probe_tma(const int32_t *ol_w, const int32_t *ol_d, const int32_
 void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id,
                        const int32_t *o_c, const int32_t *o_cnt, const int64_t *o_ent,
                        uint64_t n_o, const int32_t *c_last, int64_t having,
-                       const Q18Scratch &s, int num_sms, cudaStream_t st) {
-    q18_having_kernel<<<grid_for((n_o + kHavingUnroll - 1) / kHavingUnroll, kHavingThreads, num_sms, 8),
-                        kHavingThreads, 0, st>>>(
-        o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o, c_last, having, s);
+                       const Q18Scratch &s, int num_sms, cudaStream_t st, int unroll) {
+    if (unroll == 4)
+        q18_having_kernel<4><<<grid_for((n_o + 3) / 4, kHavingThreads, num_sms, 8), kHavingThreads, 0, st>>>(
+            o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o, c_last, having, s);
+    else
+        q18_having_kernel<2><<<grid_for((n_o + 1) / 2, kHavingThreads, num_sms, 8), kHavingThreads, 0, st>>>(
+            o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o, c_last, having, s);
     count_launches(1);
 }
 

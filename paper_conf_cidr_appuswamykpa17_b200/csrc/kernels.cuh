@@ -117,7 +117,7 @@ void launch_q18_probe_tma(const int32_t *ol_w, const int32_t *ol_d, const int32_
 void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id,
                        const int32_t *o_c, const int32_t *o_cnt, const int64_t *o_ent,
                        uint64_t n_o, const int32_t *c_last, int64_t having,
-                       const Q18Scratch &s, int num_sms, cudaStream_t st);
+                       const Q18Scratch &s, int num_sms, cudaStream_t st, int unroll = 2);
 // CH Q3 (NEXT-2) on the Q18 machinery: mark orders rows joined by new_order and an 'prefix%'
 // customer (multiplicity in acc[].pad, candidate list in cand / *ncand), probe order_line into the
 // marked rows only, emit result rows (revenue = sum x multiplicity, count *nout) + sort statistics.
