@@ -138,8 +138,8 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes):
         "q18_sort_keys_hist": (32 + 8 + 8 + 4) * n_pass,   # rows + amounts -> keys + row ids
         # ORDER BY v2 (default): count matrix + scatter computing keys + chunked local sort
         "q18_sort_hist": 8 * n_pass,                       # amounts (bucket bits inside field a)
-        "q18_bucket_scatter": (40 + 12) * n_pass if sort_passes == "v2" else (12 + 12) * n_pass,
-        "q18_bucket_sort_emit": (12 + 32 + 40) * n_pass,   # (key, id), row gather, 8 result columns
+        "q18_bucket_scatter": (40 + 16) * n_pass if sort_passes == "v2" else (12 + 12) * n_pass,
+        "q18_bucket_sort_emit": (16 if sort_passes == "v2" else 12) * n_pass + (32 + 40) * n_pass,
     }.get(kernel)
 
 

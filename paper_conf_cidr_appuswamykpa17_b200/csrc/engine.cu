@@ -1058,6 +1058,7 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
                          &marks);
     } else {
         bs.mat = static_cast<unsigned int *>(e->arena.get("q18.bmat", 4ull * ob_grid(e->num_sms) << kBucketMaxBits));
+        bs.kv = static_cast<unsigned long long *>(e->arena.get("q18.kv", 16 * n_max));
         q18_bucket_order_v2(q.rows, q.amt, q.plan_dev, n_max, bb, bs, d, q.tie_dev, e->num_sms, e->compute,
                             &marks);
     }

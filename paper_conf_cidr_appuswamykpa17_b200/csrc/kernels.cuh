@@ -163,6 +163,7 @@ struct BucketSort {
     unsigned int *big;     // [1 + 2^kBucketMaxBits]: count, then ids of buckets > small capacity
     unsigned int *ticket;  // [1], zero-initialised once, self-resetting
     unsigned int *mat;     // v2: [ob_grid * 2^bucket_bits] per-partition bucket counts -> offsets
+    unsigned long long *kv;// v2: [2 n] interleaved (key, row id) pairs in bucket order
 };
 // Optional per-kernel profiling marks (the engine records CUDA events around each phase).
 struct PhaseMarks {

@@ -477,7 +477,8 @@ template <int kLsCap> struct LsSmem {
 // inside its sub-bucket, order equal-prefix runs by the full tuple, and write the result columns
 // at their final positions. The small instance walks every bucket and queues buckets above its
 // capacity in big[1..]; the large instance walks only that queue.
-template <int kLsCap, int kMin>
+// kPairs: k holds interleaved 16-byte (key, row id) pairs (v2 scatter), v is unused.
+template <int kLsCap, int kMin, bool kPairs = false>
 __global__ void __launch_bounds__(kBkThreads)
 bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigned int *__restrict__ v,
                          const unsigned int *__restrict__ offset, int nb,
@@ -505,7 +506,10 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
             continue;
         }
         if (m == 1) {
-            if (threadIdx.x == 0) { S.k1[0] = k[lo]; S.v1[0] = v[lo]; }
+            if (threadIdx.x == 0) {
+                if (kPairs) { S.k1[0] = k[2ull * lo]; S.v1[0] = (unsigned int)k[2ull * lo + 1]; }
+                else { S.k1[0] = k[lo]; S.v1[0] = v[lo]; }
+            }
         } else {
             // sub-bucket bits: ~8 rows per sub-bucket, at most kLsSubMax sub-buckets
             int sb = 0;
@@ -521,7 +525,16 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
 #pragma unroll
                 for (int u = 0; u < 2; ++u) {
                     const unsigned int i = i0 + u * kBkThreads;
-                    if (i < m) { kk[u] = __ldcs(k + lo + i); vv[u] = __ldcs(v + lo + i); }
+                    if (i < m) {
+                        if (kPairs) {
+                            const ulonglong2 kv = __ldcs(reinterpret_cast<const ulonglong2 *>(k) + lo + i);
+                            kk[u] = kv.x;
+                            vv[u] = (unsigned int)kv.y;
+                        } else {
+                            kk[u] = __ldcs(k + lo + i);
+                            vv[u] = __ldcs(v + lo + i);
+                        }
+                    }
                 }
 #pragma unroll
                 for (int u = 0; u < 2; ++u) {
@@ -647,7 +660,8 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
 //  2. ob_scan:    per bucket, exclusive scan down the [G][nb] matrix column (staged through
 //                 shared memory); the last block scans the bucket totals into bucket offsets;
 //  3. ob_scatter: block b seeds shared cursors with offset[j] + matrix[b][j] — no global atomics —
-//                 recomputes every key from the row and writes (key, row id) at its position;
+//                 recomputes every key from the row and writes the 16-byte (key, row id) pair at
+//                 its position (one scattered store per row);
 //  4. v1's per-bucket shared-memory sort + tie-fix + emit on the (key, row id) pairs.
 // Measured and rejected: carrying the 32-byte rows through the scatter (the
 // scattered 40 B/row writes cost more than the random gather they save) and sorting chunks of
@@ -779,8 +793,7 @@ ob_scan_kernel(unsigned int *__restrict__ mat, int G, int nb, unsigned int *__re
 __global__ void __launch_bounds__(kObThreads)
 ob_scatter_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
                   const Q18Plan *__restrict__ plan, int nb, const unsigned int *__restrict__ mat,
-                  const unsigned int *__restrict__ offset, unsigned long long *__restrict__ kout,
-                  unsigned int *__restrict__ vout) {
+                  const unsigned int *__restrict__ offset, unsigned long long *__restrict__ kvout) {
     extern __shared__ unsigned int cur[];
     const uint64_t n = plan->n;
     const Q18SortSpec sp = plan->spec;
@@ -811,8 +824,7 @@ ob_scatter_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__
             if (i >= r1) break;
             const unsigned long long kk = prefix_key(r[u], a[u], sp);
             const unsigned int p = atomicAdd(&cur[(unsigned int)(kk >> shift)], 1u);
-            kout[p] = kk;
-            vout[p] = (unsigned int)i;
+            reinterpret_cast<ulonglong2 *>(kvout)[p] = make_ulonglong2(kk, (unsigned long long)i);
         }
     }
 }
@@ -891,9 +903,9 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
     const int G = ob_grid(num_sms);
     static bool init = false;
     if (!init) {
-        cudaFuncSetAttribute(bucket_local_emit_kernel<kObCap, 0>,
+        cudaFuncSetAttribute(bucket_local_emit_kernel<kObCap, 0, true>,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kObCap>));
-        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapLarge, kObCap>,
+        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>,
                              cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapLarge>));
         cudaFuncSetAttribute(ob_hist_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 << kBucketMaxBits);
         cudaFuncSetAttribute(ob_scatter_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 << kBucketMaxBits);
@@ -913,20 +925,20 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
     count_launches(1);
     end();
     begin("q18_bucket_scatter");
-    ob_scatter_kernel<<<G, kObThreads, nb * 4, st>>>(rows, amt, plan, nb, s.mat, s.offset, s.k[0], s.v[0]);
+    ob_scatter_kernel<<<G, kObThreads, nb * 4, st>>>(rows, amt, plan, nb, s.mat, s.offset, s.kv);
     count_launches(1);
     end();
     // per-bucket shared-memory sort + tie-fix + emit: the v1 kernels on the (key, row id) pairs
     begin("q18_bucket_sort_emit");
     const unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
-    bucket_local_emit_kernel<kObCap, 0><<<lb, kBkThreads, sizeof(LsSmem<kObCap>), st>>>(
-        s.k[0], s.v[0], s.offset, nb, plan, rows, amt, dst, flag, s.big);
+    bucket_local_emit_kernel<kObCap, 0, true><<<lb, kBkThreads, sizeof(LsSmem<kObCap>), st>>>(
+        s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
     end();
     begin("q18_bucket_sort_emit_large");
-    bucket_local_emit_kernel<kLsCapLarge, kObCap><<<(unsigned)num_sms, kBkThreads,
-                                                          sizeof(LsSmem<kLsCapLarge>), st>>>(
-        s.k[0], s.v[0], s.offset, nb, plan, rows, amt, dst, flag, s.big);
+    bucket_local_emit_kernel<kLsCapLarge, kObCap, true><<<(unsigned)num_sms, kBkThreads,
+                                                                sizeof(LsSmem<kLsCapLarge>), st>>>(
+        s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
     end();
 }

@@ -1,0 +1,91 @@
+#!/usr/bin/env python
+"""Config C4 on ONE B200: CH Q1 + Q6 at W=1000 (~300 M order_line rows, 7.2 GB / 6.0 GB of scanned
+columns) resident in HBM — the whole C4 dataset fits one GPU's 180 GB, so the per-GPU kernels of
+the 2/4/8-GPU runs are measured here at 1x, 8x the bench's shard. Results are checked against the
+CPU oracle on the same rows (bit-exact sums / counts, AVG rel 1e-9), then each query is timed with
+CUDA events on the engine stream (median of K, L2 irrelevant: 6-7 GB per scan).
+
+Usage: python scripts/c4_one_gpu.py [--warehouses 1000] [--steps 10] [--out F]
+"""
+import argparse
+import json
+import os
+import sys
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+import chgen  # noqa: E402
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--warehouses", type=int, default=1000)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--out", default=None)
+    a = ap.parse_args()
+    import torch
+    import oracle
+    import paper_conf_cidr_appuswamykpa17_b200 as h
+    t0 = time.time()
+    # generate in slices (bounded peak memory), keep only the Q1/Q6 columns
+    cols = ["ol_number", "ol_delivery_d", "ol_quantity", "ol_amount"]
+    parts = []
+    for lo in range(1, a.warehouses + 1, 50):
+        g = chgen.generate(lo, min(lo + 50, a.warehouses + 1), seed=1, with_item=False)
+        parts.append({c: g["order_line"][c] for c in cols})
+    ol = {c: np.concatenate([p[c] for p in parts]) for c in cols}
+    del parts
+    n = len(ol["ol_amount"])
+    gen_s = time.time() - t0
+    q6p = [chgen.ts_us("1999-01-01"), chgen.ts_us("2020-01-01"), 1, 100000]
+    q1p = [chgen.ts_us("2007-01-02")]
+    e = h.h2tap_open(0)
+    h.h2tap_load_snapshot(e, {"order_line": ol}, 1)
+    # parity against the oracle on the full 300 M rows
+    t1 = time.time()
+    w6 = oracle.q6({"order_line": ol}, *q6p)
+    w1 = oracle.q1({"order_line": ol}, *q1p)
+    oracle_s = time.time() - t1
+    r = h.h2tap_run_query(e, h.H2TAP_Q6, q6p); g6 = r.to_numpy(); r.free()
+    assert int(g6["revenue"][0]) == w6["revenue"] and int(g6["count_rows"][0]) == w6["count"]
+    r = h.h2tap_run_query(e, h.H2TAP_Q1, q1p); g1 = r.to_numpy(); r.free()
+    for k in ("ol_number", "sum_qty", "sum_amount", "count_order"):
+        assert np.array_equal(g1[k], w1[k]), k
+    for k in ("avg_qty", "avg_amount"):
+        assert np.allclose(g1[k], w1[k], rtol=1e-9, atol=0), k
+    stream = torch.cuda.ExternalStream(h.h2tap_compute_stream(e))
+    peaks = json.load(open(os.path.join(ROOT, "MEASURED_PEAKS.json"))) \
+        if os.path.exists(os.path.join(ROOT, "MEASURED_PEAKS.json")) else {}
+    peak = peaks.get("hbm_gbs", 6650.0)
+    out = {}
+    for name, plan, p, bpr in (("q6", h.H2TAP_Q6, q6p, 20), ("q1", h.H2TAP_Q1, q1p, 24)):
+        ms = []
+        for i in range(a.steps + 3):
+            torch.cuda.synchronize()
+            with torch.cuda.stream(stream):
+                b, en = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                b.record(stream)
+                rr = h.h2tap_run_query(e, plan, p, flags=h.H2TAP_RESULT_DEVICE)
+                en.record(stream)
+            torch.cuda.synchronize()
+            h.h2tap_free(rr)
+            if i >= 3:
+                ms.append(b.elapsed_time(en))
+        med = float(np.median(ms))
+        gbs = bpr * n / (med * 1e-3) / 1e9
+        out[name] = {"ms_median": round(med, 4), "rows_per_s": n / (med * 1e-3), "GBps": round(gbs, 1),
+                     "frac_of_peak": round(gbs / peak, 3)}
+    h.h2tap_close(e)
+    line = {"what": "config C4 (Q1 + Q6, W=1000) on one B200, snapshot resident, parity vs oracle passed",
+            "warehouses": a.warehouses, "order_line_rows": n, "peak_GBps": peak, "generate_s": round(gen_s, 1),
+            "oracle_s_q6_plus_q1": round(oracle_s, 1), "oracle_rows_per_s": 2 * n / oracle_s, "queries": out}
+    print(json.dumps(line))
+    if a.out:
+        open(a.out, "w").write(json.dumps(line) + "\n")
+
+
+if __name__ == "__main__":
+    main()
