@@ -67,6 +67,9 @@ if traffic:
              "ob_hist_kernel": "q18_sort_hist", "ob_scan_kernel": "q18_sort_scan",
              "ob_scatter_kernel": "q18_bucket_scatter", "ob_local_emit_kernel<2048, 0>": "q18_bucket_sort_emit",
              "ob_local_emit_kernel<8192, 2048>": "q18_bucket_sort_emit_large",
+             "q18_probe_kernel<0>": "q18_probe_groupjoin", "q18_having_kernel<2>": "q18_having_compact",
+             "bucket_local_emit_kernel<2048, 0, 1>": "q18_bucket_sort_emit",
+             "bucket_local_emit_kernel<8192, 2048, 1>": "q18_bucket_sort_emit_large",
              "q18_plan_kernel": "q18_plan", "q1_compact_kernel": "q1_compact",
              "q1_emit_kernel": "q1_emit"}
     bymark = {}
