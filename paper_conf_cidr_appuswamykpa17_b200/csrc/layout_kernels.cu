@@ -85,6 +85,7 @@ dsm_sum_kernel(const int32_t *__restrict__ data, uint64_t stride, uint64_t n, La
 // sequence of (page, selected minipage) pairs q = page * N + j; a warp step covers
 // mps = 32 / (mp_rows / 4) consecutive pairs (one 16-byte vector per lane; kUnroll steps in
 // flight), so only selected minipages are read — whole sectors — and no lane idles for any N.
+// (page, j) is carried incrementally (divisions by N only once per thread, none per vector).
 __global__ void __launch_bounds__(kThreads)
 pax_sum_kernel(const int32_t *__restrict__ data, uint64_t n, int log_ncols, int log_mp, LayoutSel sel,
                unsigned long long *out) {
@@ -94,24 +95,32 @@ pax_sum_kernel(const int32_t *__restrict__ data, uint64_t n, int log_ncols, int 
     const int mps = vpm >= 32 ? 1 : 32 / vpm;                 // pairs per warp step
     const int sub = vpm >= 32 ? 0 : lane >> log_vpm;          // this lane's pair in the step
     const uint64_t pages = (n + (1ull << log_mp) - 1) >> log_mp;
-    const unsigned total = (unsigned)(pages * (uint64_t)sel.n);  // < 2^32 (host check)
-    const unsigned N = (unsigned)sel.n;
+    const uint64_t N = (uint64_t)sel.n;
     const uint64_t gwarp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
     const uint64_t wstep = (uint64_t)mps * kUnroll;           // pairs per warp iteration
+    // iteration base q0 = gwarp * wstep as (p0, j0); stride nwarps * wstep as (sp, sj)
+    uint64_t p0 = (gwarp * wstep) / N, j0 = (gwarp * wstep) % N;
+    const uint64_t S = nwarps * wstep, sp = S / N, sj = S % N;
+    uint64_t dp[kUnroll], dj[kUnroll];                        // offsets u * mps + sub as (page, j)
+#pragma unroll
+    for (int u = 0; u < kUnroll; ++u) {
+        const uint64_t off = (uint64_t)u * mps + sub;
+        dp[u] = off / N;
+        dj[u] = off % N;
+    }
     long long acc = 0;
-    for (uint64_t qb = gwarp * wstep; qb < total; qb += nwarps * wstep) {
+    for (; p0 < pages;) {
         for (int v0 = 0; v0 < vpm; v0 += 32) {                 // minipages wider than a warp
             const int v = vpm >= 32 ? v0 + lane : (lane & (vpm - 1));
             int4 x[kUnroll];
             unsigned sel4[kUnroll];
 #pragma unroll
             for (int u = 0; u < kUnroll; ++u) {
-                const uint64_t q = qb + (uint64_t)u * mps + sub;
+                uint64_t p = p0 + dp[u], j = j0 + dj[u];
+                if (j >= N) { j -= N; ++p; }
                 sel4[u] = 0;
-                if (q < total) {
-                    const unsigned page32 = (unsigned)q / N, j = (unsigned)q - page32 * N;
-                    const uint64_t p = page32;
+                if (p < pages) {
                     const uint64_t row0 = (p << log_mp) + 4 * (uint64_t)v;
                     sel4[u] = row0 >= n ? 0u : (n - row0 >= 4 ? 0xfu : (1u << (unsigned)(n - row0)) - 1u);
                     const uint64_t off = (((p << log_ncols) + (unsigned)sel.col[j]) << log_mp) + 4 * (uint64_t)v;
@@ -122,6 +131,9 @@ pax_sum_kernel(const int32_t *__restrict__ data, uint64_t n, int log_ncols, int 
             for (int u = 0; u < kUnroll; ++u)
                 if (sel4[u]) acc += lanes_sum(x[u], sel4[u]);
         }
+        p0 += sp;
+        j0 += sj;
+        if (j0 >= N) { j0 -= N; ++p0; }
     }
     block_add(acc, out);
 }
