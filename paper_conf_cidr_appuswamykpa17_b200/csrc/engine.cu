@@ -794,6 +794,7 @@ struct QueryCtx {
     cudaEvent_t begin = nullptr, end = nullptr;
     uint64_t launches0 = 0, launches = 0;
     std::pair<void *, size_t> small{};     // pinned scalars read back at finish
+    void *small_dev = nullptr;             // its mapped device address: kernels write it directly
     std::chrono::steady_clock::time_point t0;
     size_t mark0 = 0, mark1 = 0;           // this query's profile marks [mark0, mark1)
     // Q1
@@ -812,6 +813,7 @@ struct QueryCtx {
     unsigned int *tie_dev = nullptr;
     bool q18_sorted_on_host_sync = false;   // world > 1 path already knows nout
     uint64_t nout_host = 0;
+    long long *q6_out = nullptr;           // Q6 result {revenue, count} on the device
     // NEXT-2: Q14 / Q12 / Q4
     Q14Scratch q14{};
     SmallGroups sg{};
@@ -841,7 +843,12 @@ void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     const int mb = q6_max_blocks(e->num_sms);
     s.block_part = static_cast<long long *>(e->arena.get("q6.part", sizeof(long long) * 2 * mb));
     s.done_counter = static_cast<unsigned int *>(e->arena.get("q6.counter", 64, true, e->compute));
-    s.out = static_cast<long long *>(e->arena.get("q6.out", 64));
+    // world == 1: the kernel writes {revenue, count} straight into the result's device block and
+    // into the mapped pinned scalars (no copies); world > 1: allreduce, then one D2H copy
+    s.out = e->world > 1 ? static_cast<long long *>(e->arena.get("q6.out", 64))
+                         : static_cast<long long *>(dev_block(e, q, 16));
+    s.host_out = e->world > 1 ? nullptr : static_cast<long long *>(q.small_dev);
+    q.q6_out = s.out;
     e->prof.run("q6_scan_filter_sum", [&] {
         (e->scan_tma && (e->zc_tma || !v.any_host(T, {H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT})) ? launch_q6_tma : launch_q6)(
             colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D), colp<int32_t>(v, T, H2TAP_OL_QUANTITY),
@@ -853,7 +860,7 @@ void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
         e->prof.run("q6_allreduce", [&] {
             NK(ncclAllReduce(s.out, s.out, 2, ncclInt64, ncclSum, e->comm, e->compute));
         });
-    CK(cudaMemcpyAsync(q.small.first, s.out, 16, cudaMemcpyDeviceToHost, e->compute));
+    if (e->world > 1) CK(cudaMemcpyAsync(q.small.first, s.out, 16, cudaMemcpyDeviceToHost, e->compute));
 }
 
 void finish_q6(h2tap_engine *e, QueryCtx &q) {
@@ -861,10 +868,16 @@ void finish_q6(h2tap_engine *e, QueryCtx &q) {
     const long long *sm = static_cast<const long long *>(q.small.first);
     const long long rev = sm[0], cnt = sm[1];
     r->nrows = 1;
-    auto *blk = static_cast<long long *>(result_block(r, 16));
-    if (r->on_device) CK(cudaMemcpy(blk, sm, 16, cudaMemcpyHostToDevice));
-    else { blk[0] = rev; blk[1] = cnt; }
-    (void)e;
+    long long *blk;
+    if (r->on_device && e->world == 1) {  // the kernel wrote the result column already
+        blk = q.q6_out;
+        give_blocks_to_result(q);
+    } else {
+        blk = static_cast<long long *>(result_block(r, 16));
+        if (r->on_device) CK(cudaMemcpy(blk, sm, 16, cudaMemcpyHostToDevice));
+        else { blk[0] = rev; blk[1] = cnt; }
+        release_dev_blocks(e, q);
+    }
     add_col(r, "revenue", H2TAP_I64, blk);
     r->null_store.back().assign(1, cnt == 0 ? 1 : 0);  // SUM over no rows IS NULL (R8)
     add_col(r, "count_rows", H2TAP_I64, blk + 1);
@@ -919,10 +932,8 @@ void launch_q1_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
             launch_q1_compact(s, e->compute);
         });
     }
+    s.host_small = static_cast<unsigned long long *>(q.small_dev);  // emit writes {ngroups, flags}
     e->prof.run("q1_emit", [&] { launch_q1_emit(s, kQ1MaxGroups, e->compute); });
-    auto *sm = static_cast<unsigned long long *>(q.small.first);
-    CK(cudaMemcpyAsync(sm, s.ngroups, 8, cudaMemcpyDeviceToHost, e->compute));
-    CK(cudaMemcpyAsync(sm + 1, s.flags, 4, cudaMemcpyDeviceToHost, e->compute));
 }
 
 void finish_q1(h2tap_engine *e, QueryCtx &q) {
@@ -1024,8 +1035,7 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     bs.offset = static_cast<unsigned int *>(e->arena.get("q18.boffset", 4 * ((1 << kBucketMaxBits) + 1)));
     bs.big = static_cast<unsigned int *>(e->arena.get("q18.bbig", 4 * ((1 << kBucketMaxBits) + 1)));
     bs.ticket = static_cast<unsigned int *>(e->arena.get("q18.bticket", 64, true, e->compute));
-    q.tie_dev = static_cast<unsigned int *>(e->arena.get("q18.tie", 64));
-    CK(cudaMemsetAsync(q.tie_dev, 0, 4, e->compute));
+    q.tie_dev = q.q18.tie;  // zeroed by q18_init / q3_init
     Q18Cols &d = q.out;
     d.c_last = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
     d.c_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
@@ -1085,6 +1095,7 @@ void q18_scratch(h2tap_engine *e, const View &v, QueryCtx &q, uint64_t rows_cap)
     s.ncand = nullptr;
     s.qbits = nullptr;
     s.qwords = 0;
+    s.tie = static_cast<unsigned int *>(e->arena.get("q18.tie", 64));  // zeroed by the init kernel
     q.r->plan_flags = (s.jo.dense ? 1u : 0u) | (s.jc.dense ? 2u : 0u);
 }
 
@@ -1191,9 +1202,8 @@ void q18_gather_and_order(h2tap_engine *e, QueryCtx &q, uint64_t n_rows_max) {
         launch_q18_stats(all, all_amt, total, s, e->num_sms, e->compute);  // stats of gathered rows
     }
     q18_sort_and_emit(e, q);
-    CK(cudaMemcpyAsync(&sm->nout, s.nout, 8, cudaMemcpyDeviceToHost, e->compute));
-    CK(cudaMemcpyAsync(&sm->err, s.err, 4, cudaMemcpyDeviceToHost, e->compute));
-    CK(cudaMemcpyAsync(&sm->tie, q.tie_dev, 4, cudaMemcpyDeviceToHost, e->compute));
+    launch_q18_publish(s.nout, s.err, q.tie_dev, q.small_dev, e->compute);  // -> sm (mapped)
+    (void)sm;
 }
 
 // ---- NEXT-2: CH Q3 (customer ⋈ new_order ⋈ orders ⋈ order_line) on the Q18 machinery
@@ -1613,6 +1623,7 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
             if (scratch_group(ctx[j].plan) == scratch_group(q.plan)) { finish_upto(i); break; }
         q.r.reset(new_result(e, *v, q.flags & H2TAP_RESULT_DEVICE));
         q.small = e->host_pool->get(256);
+        CK(cudaHostGetDevicePointer(&q.small_dev, q.small.first, 0));
         if (!q.begin) {
             q.begin = e->prof.ev();
             q.end = e->prof.ev();

@@ -48,6 +48,7 @@ __global__ void q18_init_kernel(Q18Scratch s) {
         *s.err = 0;
         *s.nout = 0;
         if (s.ncand) *s.ncand = 0;
+        if (s.tie) *s.tie = 0;
         Q18Stats st;
         st.amt_min = INT64_MAX; st.amt_max = INT64_MIN; st.ent_min = INT64_MAX; st.ent_max = INT64_MIN;
         st.w_min = INT32_MAX; st.w_max = INT32_MIN; st.d_min = INT32_MAX; st.d_max = INT32_MIN;
@@ -574,7 +575,21 @@ q3_emit_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
     stat.flush(s.stat_part, s.ticket, s.stats);
 }
 
+struct Q18SmallDev { unsigned long long nout; unsigned int err, tie; };  // = engine's Q18Small head
+__global__ void q18_publish_kernel(const unsigned long long *nout, const unsigned int *err,
+                                   const unsigned int *tie, Q18SmallDev *out) {
+    out->nout = *nout;
+    out->err = *err;
+    out->tie = *tie;
+}
+
 }  // namespace
+
+void launch_q18_publish(const unsigned long long *nout, const unsigned int *err, const unsigned int *tie,
+                        void *host_small, cudaStream_t st) {
+    q18_publish_kernel<<<1, 1, 0, st>>>(nout, err, tie, static_cast<Q18SmallDev *>(host_small));
+    count_launches(1);
+}
 
 void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st) {
     (void)n_orders;

@@ -16,6 +16,7 @@ struct Q6Scratch {
     long long *block_part;      // [2 * max_blocks]
     unsigned int *done_counter; // [1], zero-initialised once at allocation
     long long *out;             // [2]
+    long long *host_out;        // [2] mapped pinned host memory (also written), or null
 };
 int q6_max_blocks(int num_sms);
 void launch_q6(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uint64_t n,
@@ -42,6 +43,7 @@ struct Q1Scratch {
     unsigned long long *ngroups; // [1]
     // output (ranked by key)
     int32_t *o_key; long long *o_qty, *o_amt, *o_cnt; double *o_avg_qty, *o_avg_amt;
+    unsigned long long *host_small;  // mapped pinned: emit writes {ngroups, flags} here, or null
 };
 void launch_q1_reset(const Q1Scratch &s, cudaStream_t st);
 void launch_q1(const int32_t *number, const int64_t *deliv, const int32_t *qty,
@@ -103,6 +105,7 @@ struct Q18Scratch {
     unsigned long long *ncand;// [1]
     unsigned int *qbits;     // [qwords] bitmap of the marked orders rows (cleared by init)
     unsigned long long qwords;
+    unsigned int *tie;       // ORDER BY flag word, zeroed by init (null: not zeroed)
 };
 void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st);
 void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
@@ -131,6 +134,9 @@ void launch_q3_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol
 void launch_q3_emit(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, const int32_t *o_c,
                     const int32_t *o_cnt, const int64_t *o_ent, uint64_t max_cand, const Q18Scratch &s,
                     int num_sms, cudaStream_t st);
+// {nout, err, tie} -> mapped pinned host memory (one launch instead of three D2H copies)
+void launch_q18_publish(const unsigned long long *nout, const unsigned int *err, const unsigned int *tie,
+                        void *host_small, cudaStream_t st);
 void launch_q18_stats(const Q18Row *rows, const long long *amt, uint64_t n, const Q18Scratch &s,
                       int num_sms, cudaStream_t st);  // recompute stats over gathered rows (multi-GPU)
 

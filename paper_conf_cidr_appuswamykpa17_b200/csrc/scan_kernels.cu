@@ -57,7 +57,7 @@ __global__ void __launch_bounds__(kQ6Threads)
 q6_kernel(const longlong2 *__restrict__ deliv, const int4 *__restrict__ qty,
           const longlong2 *__restrict__ amt, uint64_t n, Q6Pred pred,
           long long *__restrict__ part, unsigned int *__restrict__ counter,
-          long long *__restrict__ out) {
+          long long *__restrict__ out, long long *__restrict__ host_out) {
     long long sum = 0, cnt = 0;
     const uint64_t nvec = n >> 2;  // 4 rows per vector: 2x16B deliv, 16B qty, 2x16B amount
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
@@ -145,6 +145,7 @@ q6_kernel(const longlong2 *__restrict__ deliv, const int4 *__restrict__ qty,
             for (int w = 0; w < kQ6Threads / 32; ++w) { S += s_sum[w]; C += s_cnt[w]; }
             out[0] = S;
             out[1] = C;
+            if (host_out) { host_out[0] = S; host_out[1] = C; }  // mapped pinned: no D2H copy
             *counter = 0;  // self-reset for the next launch
         }
     }
@@ -170,7 +171,7 @@ __global__ void __launch_bounds__(kTmaThreads, 1)
 q6_tma_kernel(const long long *__restrict__ deliv, const int *__restrict__ qty,
               const long long *__restrict__ amt, uint64_t n, Q6Pred pred,
               long long *__restrict__ part, unsigned int *__restrict__ counter,
-              long long *__restrict__ out) {
+              long long *__restrict__ out, long long *__restrict__ host_out) {
     extern __shared__ __align__(128) unsigned char smem_raw[];
     Q6TmaSmem &S = *reinterpret_cast<Q6TmaSmem *>(smem_raw);
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
@@ -246,6 +247,7 @@ q6_tma_kernel(const long long *__restrict__ deliv, const int *__restrict__ qty,
         if (lane == 0) {
             out[0] = ts;
             out[1] = tc;
+            if (host_out) { host_out[0] = ts; host_out[1] = tc; }
             *counter = 0;
         }
     }
@@ -579,6 +581,10 @@ __global__ void q1_merge_kernel(const Q1Group *__restrict__ all, uint64_t n, Q1S
 __global__ void q1_emit_kernel(Q1Scratch g) {
     __shared__ long long tile[1024];
     const uint64_t ng = *g.ngroups;  // read on the device: no host round trip before emitting
+    if (g.host_small && blockIdx.x == 0 && threadIdx.x == 0) {  // mapped pinned: no D2H copies
+        g.host_small[0] = ng;
+        reinterpret_cast<unsigned int *>(g.host_small)[2] = *g.flags;
+    }
     if ((uint64_t)blockIdx.x * blockDim.x >= ng) return;  // grid sized for the maximum
     const uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
     const long long mine = i < ng ? g.groups[i].key : 0;
@@ -619,7 +625,7 @@ void launch_q6(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uin
     q6_kernel<<<(unsigned)grid, kQ6Threads, 0, st>>>(
         reinterpret_cast<const longlong2 *>(deliv), reinterpret_cast<const int4 *>(qty),
         reinterpret_cast<const longlong2 *>(amt), n, Q6Pred{d_lo, d_hi, q_lo, q_hi},
-        s.block_part, s.done_counter, s.out);
+        s.block_part, s.done_counter, s.out, s.host_out);
         count_launches(1);
 }
 
@@ -636,7 +642,7 @@ void launch_q6_tma(const int64_t *deliv, const int32_t *qty, const int64_t *amt,
     const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
     q6_tma_kernel<<<grid, kTmaThreads, sizeof(Q6TmaSmem), st>>>(
         reinterpret_cast<const long long *>(deliv), qty, reinterpret_cast<const long long *>(amt), n,
-        Q6Pred{d_lo, d_hi, q_lo, q_hi}, s.block_part, s.done_counter, s.out);
+        Q6Pred{d_lo, d_hi, q_lo, q_hi}, s.block_part, s.done_counter, s.out, s.host_out);
     count_launches(1);
 }
 

@@ -688,8 +688,10 @@ __device__ __forceinline__ void ob_range(uint64_t n, uint64_t &r0, uint64_t &r1)
 
 __global__ void __launch_bounds__(kObThreads)
 ob_hist_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
-               const Q18Plan *__restrict__ plan, int nb, unsigned int *__restrict__ mat) {
+               const Q18Plan *__restrict__ plan, int nb, unsigned int *__restrict__ mat,
+               unsigned int *__restrict__ big) {
     extern __shared__ unsigned int h[];
+    if (blockIdx.x == 0 && threadIdx.x == 0) *big = 0;  // work-list count of the emit kernels
     const uint64_t n = plan->n;
     const Q18SortSpec sp = plan->spec;
     const int shift = plan->shift;
@@ -914,9 +916,8 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
         init = true;
     }
     (void)n_max;
-    cudaMemsetAsync(s.big, 0, sizeof(unsigned int), st);
     begin("q18_sort_hist");
-    ob_hist_kernel<<<G, kObThreads, nb * 4, st>>>(rows, amt, plan, nb, s.mat);
+    ob_hist_kernel<<<G, kObThreads, nb * 4, st>>>(rows, amt, plan, nb, s.mat, s.big);
     count_launches(1);
     end();
     begin("q18_sort_scan");
