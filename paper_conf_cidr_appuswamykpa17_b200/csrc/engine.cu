@@ -196,9 +196,21 @@ struct ResultImpl : h2tap_result {
 };
 
 // =========================================================== snapshot ===
-constexpr int kStatCols = 3;  // min/max kept for the (w, d, id) key columns 0..2 of each table
-// (item: i_id only — its columns 1..2 are not keys)
+constexpr int kStatCols = 4;  // zone-map slots per table: the (w, d, id) key columns 0..2, and
+// slot 3 = a payload column of the Q18 result rows (orders: o_ol_cnt; customer: c_last) whose
+// range sizes the ORDER BY's carry records; item: i_id only
 inline int stat_cols(int table) { return table == H2TAP_T_ITEM ? 1 : kStatCols; }
+inline int stat_col(int table, int slot) {  // column id of a zone-map slot, -1 if none
+    if (slot < 3) return slot;
+    if (table == H2TAP_T_ORDERS) return H2TAP_O_OL_CNT;
+    if (table == H2TAP_T_CUSTOMER) return H2TAP_C_LAST;
+    return -1;
+}
+inline int stat_slot(int table, uint32_t column) {  // zone-map slot of a column, -1 if none
+    for (int s = 0; s < stat_cols(table); ++s)
+        if (stat_col(table, s) == (int)column) return s;
+    return -1;
+}
 struct View {  // immutable snapshot at one epoch (the paper's shallow-copied top container)
     uint64_t epoch = 0;
     uint64_t n[kTables] = {};
@@ -656,8 +668,8 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         pend.full[t.table_id] = full;
         // zone map of the appended rows' key columns, on the copy stream after their H2D
         for (int c = 0; c < stat_cols(t.table_id); ++c)
-            if (v->col[t.table_id][c])
-                launch_minmax_i32(static_cast<const int32_t *>(v->col[t.table_id][c]) + t.first_row,
+            if (stat_col(t.table_id, c) >= 0 && v->col[t.table_id][stat_col(t.table_id, c)])
+                launch_minmax_i32(static_cast<const int32_t *>(v->col[t.table_id][stat_col(t.table_id, c)]) + t.first_row,
                                   t.row_count - t.first_row,
                                   stats_dev + (t.table_id * kStatCols + c) * 2, e->num_sms, e->copy);
     }
@@ -712,9 +724,10 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
             const auto *rows_d = reinterpret_cast<const uint32_t *>(upd_dev + upd_off[i]);
             const void *vals_d = upd_dev + upd_off[i] + round_up16(u.n * 4);
             launch_apply_updates(cs.alt->ptr, (uint32_t)es, next_bits, rows_d, vals_d, u.n, e->num_sms, e->copy);
-            if (u.column_id < (uint32_t)stat_cols(u.table_id))  // zone map: widen
+            if (stat_slot(u.table_id, u.column_id) >= 0)  // zone map: widen
                 launch_minmax_i32(static_cast<const int32_t *>(vals_d), u.n,
-                                  stats_dev + (u.table_id * kStatCols + u.column_id) * 2, e->num_sms, e->copy);
+                                  stats_dev + (u.table_id * kStatCols + stat_slot(u.table_id, u.column_id)) * 2,
+                                  e->num_sms, e->copy);
         }
         std::swap(cs.cur, cs.alt);
         std::swap(cs.bits, cs.bits_next);
@@ -803,6 +816,7 @@ struct QueryCtx {
     // Q18
     Q18Scratch q18{};
     Q18Plan *plan_dev = nullptr;
+    Q18Zone zone{};                         // ORDER BY field bounds from the zone maps
     const Q18Row *rows = nullptr;
     const long long *amt = nullptr;
     const unsigned int *perm = nullptr;
@@ -1021,7 +1035,12 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     if (const char *d = std::getenv("H2TAP_BUCKET_BITS_DELTA"))      // tuning knob
         bb = std::max(1, std::min(kBucketMaxBits, bb + std::atoi(d)));
     q.plan_dev = static_cast<Q18Plan *>(e->arena.get("q18.plan", sizeof(Q18Plan)));
-    e->prof.run("q18_plan", [&] { launch_q18_plan(q.q18.stats, q.q18.nout, bb, q.plan_dev, e->compute); });
+    // carry records unless disabled for A/B (H2TAP_ORDER_CARRY=0) or on v1
+    const char *cv = std::getenv("H2TAP_ORDER_CARRY");
+    const bool carry = !e->order_v1 && !(cv && cv[0] == '0');
+    e->prof.run("q18_plan", [&] {
+        launch_q18_plan(q.q18.stats, q.zone, q.q18.nout, bb, carry, q.plan_dev, q.q18.tie, e->compute);
+    });
     for (int b = 0; b < 2; ++b) {
         q.sp.k[b] = static_cast<unsigned long long *>(e->arena.get("q18.sk" + std::to_string(b), 8 * n_max));
         q.sp.v[b] = static_cast<unsigned int *>(e->arena.get("q18.sv" + std::to_string(b), 4 * n_max));
@@ -1101,6 +1120,23 @@ void q18_scratch(h2tap_engine *e, const View &v, QueryCtx &q, uint64_t rows_cap)
 
 void q18_gather_and_order(h2tap_engine *e, QueryCtx &q, uint64_t n_rows_max);
 
+// Bounds of the result rows' (w, d, o) and payload fields from the published zone maps: every
+// result row is an orders row matched to a customer row of this snapshot. Q3 returns no
+// customer / o_ol_cnt fields (its rows carry zeros there).
+Q18Zone q18_zone(const View &v, bool q3) {
+    const int O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
+    Q18Zone z{};
+    z.w_min = v.smin[O][0]; z.w_max = v.smax[O][0];
+    z.d_min = v.smin[O][1]; z.d_max = v.smax[O][1];
+    z.o_min = v.smin[O][2]; z.o_max = v.smax[O][2];
+    if (!q3) {
+        z.cl_min = v.smin[C][3]; z.cl_max = v.smax[C][3];
+        z.ci_min = v.smin[C][2]; z.ci_max = v.smax[C][2];
+        z.n_min = v.smin[O][3]; z.n_max = v.smax[O][3];
+    }
+    return z;
+}
+
 void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
     need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}, "Q18");
@@ -1133,6 +1169,7 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
                               e->having_unroll);
     });
     CK(cudaGetLastError());
+    q.zone = q18_zone(v, false);
     q18_gather_and_order(e, q, n_o);
 }
 
@@ -1157,6 +1194,22 @@ void q18_gather_and_order(h2tap_engine *e, QueryCtx &q, uint64_t n_rows_max) {
         sync_compute(e);
         if (sm->err) return;  // finish raises the local error
         if (err_any) raise(H2TAP_EPLAN, "Q%u: failed on another rank", q.plan);
+        {   // the ORDER BY bounds must cover every rank's rows: min/max of the zones
+            static_assert(sizeof(Q18Zone) == 12 * sizeof(int), "Q18Zone: 6 (min, max) int pairs");
+            int zmin[6], zmax[6];
+            const int *zp = reinterpret_cast<const int *>(&q.zone);
+            for (int k = 0; k < 6; ++k) { zmin[k] = zp[2 * k]; zmax[k] = zp[2 * k + 1]; }
+            auto *zd = static_cast<int *>(e->arena.get("q18.zone", 64));
+            CK(cudaMemcpyAsync(zd, zmin, 24, cudaMemcpyHostToDevice, e->compute));
+            CK(cudaMemcpyAsync(zd + 6, zmax, 24, cudaMemcpyHostToDevice, e->compute));
+            NK(ncclAllReduce(zd, zd, 6, ncclInt32, ncclMin, e->comm, e->compute));
+            NK(ncclAllReduce(zd + 6, zd + 6, 6, ncclInt32, ncclMax, e->comm, e->compute));
+            CK(cudaMemcpyAsync(zmin, zd, 24, cudaMemcpyDeviceToHost, e->compute));
+            CK(cudaMemcpyAsync(zmax, zd + 6, 24, cudaMemcpyDeviceToHost, e->compute));
+            sync_compute(e);
+            int *zw = reinterpret_cast<int *>(&q.zone);
+            for (int k = 0; k < 6; ++k) { zw[2 * k] = zmin[k]; zw[2 * k + 1] = zmax[k]; }
+        }
         auto *cnt_dev = static_cast<unsigned long long *>(e->arena.get("q18.allcnt", 8ull * e->world));
         NK(ncclAllGather(s.nout, cnt_dev, 1, ncclUint64, e->comm, e->compute));
         std::vector<unsigned long long> cnts(e->world);
@@ -1250,6 +1303,7 @@ void launch_q3_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
                            e->num_sms, e->compute);
     });
     CK(cudaGetLastError());
+    q.zone = q18_zone(v, true);
     q18_gather_and_order(e, q, cap);
 }
 
@@ -1279,10 +1333,16 @@ void finish_q18(h2tap_engine *e, QueryCtx &q) {
         Q18Plan hp;
         CK(cudaMemcpy(&hp, q.plan_dev, sizeof hp, cudaMemcpyDeviceToHost));
         launch_iota(w.v[0], nout, e->num_sms, e->compute);
-        const int fb[3] = {hp.spec.bits_r, hp.spec.bits_e, hp.spec.bits_a};
-        for (int f = 0; f < 3; ++f) {
+        // (r = the concatenated (w, d, o) fields; wider than 62 bits: o, d, w sorted one by one)
+        const bool wide = hp.spec.wide_r != 0;
+        const int fid[5] = {3, 4, 5, 1, 2};
+        const int nf = wide ? 5 : 3;
+        for (int k = 0; k < nf; ++k) {
+            const int f = wide ? fid[k] : k;
+            const int bits = f == 0 ? hp.spec.bits_r : f == 1 ? hp.spec.bits_e : f == 2 ? hp.spec.bits_a
+                           : f == 3 ? hp.spec.bits_o : f == 4 ? hp.spec.bits_d : hp.spec.bits_w;
             launch_q18_field_keys(q.rows, q.amt, w.v[0], nout, f, q.plan_dev, w.k[0], e->num_sms, e->compute);
-            const int cur = radix_sort_pairs(nout, fb[f], w, e->num_sms, e->compute);
+            const int cur = radix_sort_pairs(nout, bits, w, e->num_sms, e->compute);
             if (cur) { std::swap(w.k[0], w.k[1]); std::swap(w.v[0], w.v[1]); }
         }
         // keys are field keys, not the prefix: amounts are read from amt[]

@@ -51,8 +51,6 @@ __global__ void q18_init_kernel(Q18Scratch s) {
         if (s.tie) *s.tie = 0;
         Q18Stats st;
         st.amt_min = INT64_MAX; st.amt_max = INT64_MIN; st.ent_min = INT64_MAX; st.ent_max = INT64_MIN;
-        st.w_min = INT32_MAX; st.w_max = INT32_MIN; st.d_min = INT32_MAX; st.d_max = INT32_MIN;
-        st.o_min = INT32_MAX; st.o_max = INT32_MIN; st.pad0 = st.pad1 = 0;
         *s.stats = st;
     }
 }
@@ -301,33 +299,24 @@ __device__ __forceinline__ long long wmax64(long long v) {
     return v;
 }
 
+// Min/max of amount_sum and o_entry_d over the result rows (the other ORDER BY fields are
+// bounded by the snapshot's zone maps, Q18Zone: fewer live registers in the HAVING kernel).
 struct StatAcc {
     long long amin = INT64_MAX, amax = INT64_MIN, emin = INT64_MAX, emax = INT64_MIN;
-    int wmin = INT32_MAX, wmax = INT32_MIN, dmin = INT32_MAX, dmax = INT32_MIN;
-    int omin = INT32_MAX, omax = INT32_MIN;
-    __device__ void add(long long a, long long e, int w, int d, int o) {
+    __device__ void add(long long a, const Q18Row &r) {
         amin = a < amin ? a : amin; amax = a > amax ? a : amax;
-        emin = e < emin ? e : emin; emax = e > emax ? e : emax;
-        wmin = min(wmin, w); wmax = max(wmax, w); dmin = min(dmin, d); dmax = max(dmax, d);
-        omin = min(omin, o); omax = max(omax, o);
+        emin = r.o_entry_d < emin ? r.o_entry_d : emin; emax = r.o_entry_d > emax ? r.o_entry_d : emax;
     }
     __device__ void merge(const Q18Stats &o) {
         amin = o.amt_min < amin ? o.amt_min : amin; amax = o.amt_max > amax ? o.amt_max : amax;
         emin = o.ent_min < emin ? o.ent_min : emin; emax = o.ent_max > emax ? o.ent_max : emax;
-        wmin = min(wmin, o.w_min); wmax = max(wmax, o.w_max); dmin = min(dmin, o.d_min);
-        dmax = max(dmax, o.d_max); omin = min(omin, o.o_min); omax = max(omax, o.o_max);
     }
     __device__ void warp_reduce() {
         amin = wmin64(amin); amax = wmax64(amax); emin = wmin64(emin); emax = wmax64(emax);
-        wmin = __reduce_min_sync(kFull, wmin); wmax = __reduce_max_sync(kFull, wmax);
-        dmin = __reduce_min_sync(kFull, dmin); dmax = __reduce_max_sync(kFull, dmax);
-        omin = __reduce_min_sync(kFull, omin); omax = __reduce_max_sync(kFull, omax);
     }
     __device__ Q18Stats get() const {
         Q18Stats s;
         s.amt_min = amin; s.amt_max = amax; s.ent_min = emin; s.ent_max = emax;
-        s.w_min = wmin; s.w_max = wmax; s.d_min = dmin; s.d_max = dmax; s.o_min = omin; s.o_max = omax;
-        s.pad0 = s.pad1 = 0;
         return s;
     }
     // Block reduction into part[blockIdx.x]; the last block to finish folds every block's
@@ -453,7 +442,7 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
             st16_policy(s.rows + p, w64[0], w64[1], keep);
             st16_policy(reinterpret_cast<char *>(s.rows + p) + 16, w64[2], w64[3], keep);
             ++p;
-            stat.add(sum[u], row[u].o_entry_d, w[u], d[u], row[u].o_id);
+            stat.add(sum[u], row[u]);
         }
         __syncthreads();  // wsum / s_base reuse
     }
@@ -466,7 +455,7 @@ __global__ void q18_stats_kernel(const Q18Row *__restrict__ rows, const long lon
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
         const Q18Row r = rows[i];
-        stat.add(amt[i], r.o_entry_d, r.o_w_id, r.o_d_id, r.o_id);
+        stat.add(amt[i], r);
     }
     stat.flush(part, ticket, st);
 }
@@ -560,15 +549,15 @@ q3_emit_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
             const uint64_t p = s_base + before + x - 1;
             Q18Row row;
             row.o_entry_d = __ldg(o_ent + r);
-            row.c_last = 0;
-            row.c_id = __ldg(o_c + r);
+            row.c_last = 0;   // Q3 outputs no customer / o_ol_cnt fields: zero payload
+            row.c_id = 0;     // (its ORDER BY zone has c_last = c_id = o_ol_cnt = 0)
             row.o_id = __ldg(o_id + r);
-            row.o_ol_cnt = __ldg(o_cnt + r);
+            row.o_ol_cnt = 0;
             row.o_w_id = __ldg(o_w + r);
             row.o_d_id = __ldg(o_d + r);
             s.rows[p] = row;
             s.amt[p] = sum;
-            stat.add(sum, row.o_entry_d, row.o_w_id, row.o_d_id, row.o_id);
+            stat.add(sum, row);
         }
         __syncthreads();
     }

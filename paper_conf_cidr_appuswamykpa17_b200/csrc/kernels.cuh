@@ -77,9 +77,12 @@ struct JoinIndex {
     unsigned int nw, nd, nk;                          // dense: box extents
     unsigned long long range;                         // dense: nw * nd * nk
 };
-struct Q18Stats {            // min/max of the sort fields over result rows (atomics)
+struct Q18Stats {            // min/max of the sort fields that only the result rows know
     long long amt_min, amt_max, ent_min, ent_max;
-    int w_min, w_max, d_min, d_max, o_min, o_max, pad0, pad1;
+};
+struct Q18Zone {             // bounds of the other result-row fields: the snapshot's zone maps
+    int w_min, w_max, d_min, d_max, o_min, o_max;      // orders (w, d, o) key columns
+    int cl_min, cl_max, ci_min, ci_max, n_min, n_max;  // c_last, c_id, o_ol_cnt (carry payload)
 };
 struct __align__(16) Q18Row {  // one result row before ORDER BY: 32 B = one L2 sector per gather
     long long o_entry_d;       // (amount_sum lives in a parallel array: after the sort it is
@@ -182,9 +185,16 @@ struct PhaseMarks {
 struct Q18SortSpec {         // host-computed from Q18Stats
     long long amt_max, ent_min;
     int w_min, d_min, o_min;
-    long long nd, no;        // extents of d and o (dense row rank)
-    int bits_a, bits_e, bits_r;  // field widths: amount (desc), entry, row rank
+    int bits_w, bits_d, bits_o;  // r = (w - w_min | d - d_min | o - o_min), fields concatenated
+    int wide_r;              // bits_w + bits_d + bits_o > 62: exact per-column fallback
+    int bits_a, bits_e, bits_r;  // field widths: amount (desc), entry, (w, d, o) tie-break
     int prefix_bits;         // width of the sorted 64-bit prefix of the composite key
+    // carry mode: the 128-bit sort record (prefix, low key bits | payload)
+    // holds the whole result row, so the emit decodes instead of gathering rows.
+    int carry;               // 1 if bits_a + bits_e + bits_r + payload bits <= 128
+    int bits_low;            // key bits below the 64-bit prefix (carried in the second word)
+    int bits_cl, bits_ci, bits_n;  // payload widths: c_last, c_id, o_ol_cnt (offsets from min)
+    int cl_min, ci_min, n_min;
 };
 // Device-side plan of the ORDER BY, computed from the HAVING kernel's statistics and row count
 // (no host round trip): field widths, 64-bit prefix width, whether a tie-fix is needed, and the
@@ -195,8 +205,9 @@ struct Q18Plan {
     int tiefix;
     int shift;
 };
-void launch_q18_plan(const Q18Stats *stats, const unsigned long long *nout, int bucket_bits,
-                     Q18Plan *plan, cudaStream_t st);
+void launch_q18_plan(const Q18Stats *stats, const Q18Zone &zone, const unsigned long long *nout,
+                     int bucket_bits, bool allow_carry, Q18Plan *plan, unsigned int *flag,
+                     cudaStream_t st);
 // The whole ORDER BY: keys + histogram -> bucket scatter -> per-bucket sort, tie-fix and emit
 // into `dst` (final positions). Everything reads the row count and widths from *plan.
 // *flag: bit0 a tie run > 32 rows, bit1 a bucket > 8192 rows (caller redoes it exactly).

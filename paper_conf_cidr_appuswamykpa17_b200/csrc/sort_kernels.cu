@@ -2,8 +2,9 @@
 // (o_w_id, o_d_id, o_id) tie-break that makes the order total (R11).
 //
 // The three sort fields are mapped to unsigned integers whose widths come from the result's
-// min/max (HAVING kernel statistics): a = max - amount_sum (DESC), e = o_entry_d - min,
-// r = dense rank of (w, d, o). Their concatenation a|e|r is the exact composite key.
+// min/max (HAVING kernel statistics) and the snapshot's zone maps: a = max - amount_sum (DESC),
+// e = o_entry_d - min, r = (w, d, o) offsets as concatenated fixed-width fields. a|e|r is the
+// exact composite key.
 //  * main path: sort (top 64 bits of a|e|r, row id) pairs with a bucket sort (partition by the
 //    top key bits, bitonic sort per bucket in shared memory). If a|e|r fits 64 bits the keys are
 //    distinct and the order is exact; otherwise runs of equal 64-bit prefixes are ordered by the
@@ -163,10 +164,12 @@ __device__ __forceinline__ unsigned long long field_e(const Q18Row &r, const Q18
     return (unsigned long long)r.o_entry_d - (unsigned long long)sp.ent_min;
 }
 __device__ __forceinline__ unsigned long long field_r(const Q18Row &r, const Q18SortSpec &sp) {
+    // (w, d, o) as concatenated fixed-width fields: lexicographic order = integer order, and
+    // the carry decode is shifts and masks (no division)
     const unsigned long long w = (unsigned)(r.o_w_id - sp.w_min);
     const unsigned long long d = (unsigned)(r.o_d_id - sp.d_min);
     const unsigned long long o = (unsigned)(r.o_id - sp.o_min);
-    return (w * (unsigned long long)sp.nd + d) * (unsigned long long)sp.no + o;
+    return (w << (sp.bits_d + sp.bits_o)) | (d << sp.bits_o) | o;
 }
 
 // top `prefix_bits` bits of the concatenation (a | e | r) with widths (bits_a, bits_e, bits_r)
@@ -196,6 +199,49 @@ __device__ __forceinline__ bool row_less(const Q18Row &x, long long ax, const Q1
     return x.o_id < y.o_id;
 }
 
+// ---- carry records: 128 bits = (top 64 key bits, low key bits | payload).
+// The key K = a|e|r is unique per result row (r encodes the orders PK), so
+// comparing (hi, lo) as one 128-bit integer is the exact ORDER BY; the payload
+// (c_last, c_id, o_ol_cnt as offsets from their minima) rides in the lowest bits.
+typedef unsigned __int128 u128;
+__device__ __forceinline__ u128 shl128(u128 x, int s) { return s >= 128 ? (u128)0 : x << s; }
+__device__ __forceinline__ u128 shr128(u128 x, int s) { return s >= 128 ? (u128)0 : x >> s; }
+__device__ __forceinline__ unsigned long long lowmask(int b) { return b >= 64 ? ~0ull : (1ull << b) - 1ull; }
+__device__ __forceinline__ unsigned long long shr64(unsigned long long x, int s) { return s >= 64 ? 0ull : x >> s; }
+
+__device__ __forceinline__ ulonglong2 carry_record(const Q18Row &r, long long amount, const Q18SortSpec &sp) {
+    const u128 K = shl128((u128)field_a(amount, sp), sp.bits_e + sp.bits_r) |
+                   shl128((u128)field_e(r, sp), sp.bits_r) | (u128)field_r(r, sp);
+    const int P = sp.bits_cl + sp.bits_ci + sp.bits_n;
+    const unsigned long long pay =
+        (((unsigned long long)((unsigned)r.c_last - (unsigned)sp.cl_min) << sp.bits_ci |
+          (unsigned long long)((unsigned)r.c_id - (unsigned)sp.ci_min)) << sp.bits_n) |
+        (unsigned long long)((unsigned)r.o_ol_cnt - (unsigned)sp.n_min);
+    const unsigned long long klo = (unsigned long long)K & lowmask(sp.bits_low);
+    return make_ulonglong2((unsigned long long)shr128(K, sp.bits_low),
+                           (unsigned long long)shl128((u128)klo, P) | pay);
+}
+
+struct CarryRow { long long amount, o_entry_d; int c_last, c_id, o_id, o_ol_cnt, o_w_id, o_d_id; };
+__device__ __forceinline__ CarryRow carry_decode(unsigned long long hi, unsigned long long lo,
+                                                 const Q18SortSpec &sp) {
+    const int P = sp.bits_cl + sp.bits_ci + sp.bits_n;
+    const u128 K = shl128((u128)hi, sp.bits_low) | (u128)(unsigned long long)shr128((u128)lo, P);
+    const unsigned long long fr = (unsigned long long)K & lowmask(sp.bits_r);
+    const unsigned long long fe = (unsigned long long)shr128(K, sp.bits_r) & lowmask(sp.bits_e);
+    const unsigned long long fa = (unsigned long long)shr128(K, sp.bits_r + sp.bits_e);
+    CarryRow c;
+    c.amount = (long long)((unsigned long long)sp.amt_max - fa);
+    c.o_entry_d = (long long)((unsigned long long)sp.ent_min + fe);
+    c.o_id = (int)((unsigned)sp.o_min + (unsigned)(fr & lowmask(sp.bits_o)));
+    c.o_d_id = (int)((unsigned)sp.d_min + (unsigned)(shr64(fr, sp.bits_o) & lowmask(sp.bits_d)));
+    c.o_w_id = (int)((unsigned)sp.w_min + (unsigned)shr64(fr, sp.bits_o + sp.bits_d));
+    c.o_ol_cnt = (int)((unsigned)sp.n_min + (unsigned)(lo & lowmask(sp.bits_n)));
+    c.c_id = (int)((unsigned)sp.ci_min + (unsigned)(shr64(lo, sp.bits_n) & lowmask(sp.bits_ci)));
+    c.c_last = (int)((unsigned)sp.cl_min + (unsigned)(shr64(lo, sp.bits_n + sp.bits_ci) & lowmask(sp.bits_cl)));
+    return c;
+}
+
 constexpr int kMaxRun = 32;
 
 __global__ void field_keys_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
@@ -206,7 +252,14 @@ __global__ void field_keys_kernel(const Q18Row *__restrict__ rows, const long lo
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
         const unsigned int x = vals[i];
         const Q18Row r = rows[x];
-        k[i] = field == 0 ? field_r(r, sp) : field == 1 ? field_e(r, sp) : field_a(amt[x], sp);
+        switch (field) {  // 0 r, 1 e, 2 a; 3 o, 4 d, 5 w (r split per column when wide_r)
+            case 0: k[i] = field_r(r, sp); break;
+            case 1: k[i] = field_e(r, sp); break;
+            case 2: k[i] = field_a(amt[x], sp); break;
+            case 3: k[i] = (unsigned)(r.o_id - sp.o_min); break;
+            case 4: k[i] = (unsigned)(r.o_d_id - sp.d_min); break;
+            default: k[i] = (unsigned)(r.o_w_id - sp.w_min); break;
+        }
     }
 }
 
@@ -256,9 +309,12 @@ __global__ void permute_kernel(const Q18Row *__restrict__ rows, const long long 
 
 __device__ __forceinline__ int bitwidth_dev(unsigned long long x) { return x ? 64 - __clzll(x) : 0; }
 
-// One thread: the ORDER BY plan from the HAVING statistics (widths of a, e, r; prefix width).
-__global__ void q18_plan_kernel(const Q18Stats *__restrict__ stats, const unsigned long long *nout,
-                                int bucket_bits, Q18Plan *plan) {
+// One thread: the ORDER BY plan from the HAVING statistics (amount_sum, o_entry_d) and the
+// snapshot's zone maps (w, d, o; carry payload): widths of a, e, r, the prefix width, and
+// whether the 128-bit carry record holds the whole row.
+__global__ void q18_plan_kernel(const Q18Stats *__restrict__ stats, Q18Zone z,
+                                const unsigned long long *nout, int bucket_bits, int allow_carry,
+                                Q18Plan *plan, unsigned int *flag) {
     const Q18Stats st = *stats;
     Q18Plan p{};
     p.n = *nout;
@@ -266,16 +322,25 @@ __global__ void q18_plan_kernel(const Q18Stats *__restrict__ stats, const unsign
     if (p.n > 1) {
         sp.amt_max = st.amt_max;
         sp.ent_min = st.ent_min;
-        sp.w_min = st.w_min; sp.d_min = st.d_min; sp.o_min = st.o_min;
-        sp.nd = (long long)st.d_max - st.d_min + 1;
-        sp.no = (long long)st.o_max - st.o_min + 1;
-        const unsigned long long nw = (unsigned long long)((long long)st.w_max - st.w_min + 1);
+        sp.w_min = z.w_min; sp.d_min = z.d_min; sp.o_min = z.o_min;
+        sp.bits_w = bitwidth_dev((unsigned)z.w_max - (unsigned)z.w_min);
+        sp.bits_d = bitwidth_dev((unsigned)z.d_max - (unsigned)z.d_min);
+        sp.bits_o = bitwidth_dev((unsigned)z.o_max - (unsigned)z.o_min);
         sp.bits_a = bitwidth_dev((unsigned long long)st.amt_max - (unsigned long long)st.amt_min);
         sp.bits_e = bitwidth_dev((unsigned long long)st.ent_max - (unsigned long long)st.ent_min);
-        sp.bits_r = bitwidth_dev(nw * (unsigned long long)sp.nd * (unsigned long long)sp.no - 1);
+        // (the join-key domain, w < 2^23, d < 2^8, o >= 0, keeps this <= 62; guard anyway)
+        sp.wide_r = sp.bits_w + sp.bits_d + sp.bits_o > 62;
+        if (sp.wide_r) atomicOr(flag, 4u);  // the engine redoes the ORDER BY per column
+        sp.bits_r = sp.wide_r ? 62 : sp.bits_w + sp.bits_d + sp.bits_o;
         const int B = sp.bits_a + sp.bits_e + sp.bits_r;
         sp.prefix_bits = B <= 64 ? B : 64;
-        p.tiefix = B > 64;
+        sp.bits_low = B - sp.prefix_bits;
+        sp.cl_min = z.cl_min; sp.ci_min = z.ci_min; sp.n_min = z.n_min;
+        sp.bits_cl = bitwidth_dev((unsigned)z.cl_max - (unsigned)z.cl_min);
+        sp.bits_ci = bitwidth_dev((unsigned)z.ci_max - (unsigned)z.ci_min);
+        sp.bits_n = bitwidth_dev((unsigned)z.n_max - (unsigned)z.n_min);
+        sp.carry = allow_carry && !sp.wide_r && sp.bits_low + sp.bits_cl + sp.bits_ci + sp.bits_n <= 64;
+        p.tiefix = B > 64 && !sp.carry;  // carry records compare all key bits: no tie-fix
         p.shift = sp.prefix_bits > bucket_bits ? sp.prefix_bits - bucket_bits : 0;
     }
     *plan = p;
@@ -290,9 +355,10 @@ unsigned grid_cap(uint64_t work, int threads, int num_sms, int per_sm) {
 
 }  // namespace
 
-void launch_q18_plan(const Q18Stats *stats, const unsigned long long *nout, int bucket_bits,
-                     Q18Plan *plan, cudaStream_t st) {
-    q18_plan_kernel<<<1, 1, 0, st>>>(stats, nout, bucket_bits, plan);
+void launch_q18_plan(const Q18Stats *stats, const Q18Zone &zone, const unsigned long long *nout,
+                     int bucket_bits, bool allow_carry, Q18Plan *plan, unsigned int *flag,
+                     cudaStream_t st) {
+    q18_plan_kernel<<<1, 1, 0, st>>>(stats, zone, nout, bucket_bits, allow_carry ? 1 : 0, plan, flag);
     count_launches(1);
 }
 
@@ -473,6 +539,151 @@ template <int kLsCap> struct LsSmem {
     unsigned int wsum[kBkThreads / 32];
 };
 
+// carry mode: 64-bit second words instead of 32-bit row ids (2 048 rows: 72 KB, 3 blocks/SM)
+template <int kCap> struct LcSmem {
+    unsigned long long k1[kCap], k2[kCap], v1[kCap], v2[kCap];
+    unsigned int sub[kLsSubMax + 1];
+    unsigned int cur[kLsSubMax];
+    unsigned int wsum[kBkThreads / 32];
+};
+constexpr int kLcCapLarge = 6144;  // carry records per bucket in the large instance (~197 KB)
+
+// Per-bucket sort of carry records (same sub-bucket + rank scheme as the row-id body below,
+// 128-bit compares, no tie-fix) and the emit: every output column is decoded from the record,
+// so the only global traffic is the bucket's records in and the result columns out. The next
+// bucket's first kPre * 256 records are loaded into registers while the current one is
+// decoded and stored, and its sub-bucket counters are cleared then too (one barrier less).
+constexpr int kPre = 2;
+template <int kCap, int kMin>
+__device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ kv,
+                                                const unsigned int *__restrict__ offset, int nb,
+                                                const Q18Plan *__restrict__ plan, const Q18Cols &dst,
+                                                unsigned int *flag, unsigned int *big, unsigned char *smem) {
+    LcSmem<kCap> &S = *reinterpret_cast<LcSmem<kCap> *>(smem);
+    const int shift = plan->shift;
+    const Q18SortSpec sp = plan->spec;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const int nwork = kMin > 0 ? (int)*(volatile unsigned int *)big : nb;
+    // bucket `wi` of this block: its range and the first kPre records of this thread
+    unsigned int lo = 0, m = 0;
+    ulonglong2 pre[kPre];
+    auto fetch = [&](int wi) {
+        lo = m = 0;
+        if (wi >= nwork) return;
+        const int b = kMin > 0 ? (int)big[1 + wi] : wi;
+        lo = offset[b];
+        m = offset[b + 1] - lo;
+        if (m == 0) return;
+        if (m > (unsigned)kCap) {
+            if (threadIdx.x == 0) {
+                if (kMin > 0) atomicOr(flag, 2u);                 // too big even for shared memory
+                else big[1 + atomicAdd(big, 1u)] = (unsigned)b;   // hand over to the large instance
+            }
+            m = 0;
+            return;
+        }
+#pragma unroll
+        for (int u = 0; u < kPre; ++u) {
+            const unsigned int i = threadIdx.x + u * kBkThreads;
+            if (i < m) pre[u] = __ldcs(kv + lo + i);
+        }
+    };
+    for (unsigned int i = threadIdx.x; i <= kLsSubMax; i += kBkThreads) S.sub[i] = 0;
+    fetch(blockIdx.x);
+    __syncthreads();
+    for (int wi = blockIdx.x; wi < nwork; wi += gridDim.x) {
+        if (m == 0) {  // empty or handed over (uniform across the block)
+            fetch(wi + gridDim.x);
+            continue;
+        }
+        int sb = 0;
+        while (sb < 10 && (m >> (sb + 3)) > 0) ++sb;
+        if (sb > shift) sb = shift;
+        const int ssh = shift - sb;
+        const unsigned int ns = 1u << sb, smask = ns - 1u;
+#pragma unroll
+        for (int u = 0; u < kPre; ++u) {
+            const unsigned int i = threadIdx.x + u * kBkThreads;
+            if (i < m) {
+                S.k1[i] = pre[u].x;
+                S.v1[i] = pre[u].y;
+                atomicAdd(&S.sub[(unsigned int)(pre[u].x >> ssh) & smask], 1u);
+            }
+        }
+        for (unsigned int i = threadIdx.x + kPre * kBkThreads; i < m; i += kBkThreads) {  // rest
+            const ulonglong2 r = __ldcs(kv + lo + i);
+            S.k1[i] = r.x;
+            S.v1[i] = r.y;
+            atomicAdd(&S.sub[(unsigned int)(r.x >> ssh) & smask], 1u);
+        }
+        __syncthreads();
+        {   // exclusive scan of ns (<= 1024) sub-bucket counts: 4 per thread
+            unsigned int c[4], t = 0;
+#pragma unroll
+            for (int q = 0; q < 4; ++q) {
+                const unsigned int i = threadIdx.x * 4 + q;
+                c[q] = i < ns ? S.sub[i] : 0u;
+                t += c[q];
+            }
+            unsigned int x = t;
+#pragma unroll
+            for (int o = 1; o < 32; o <<= 1) {
+                const unsigned int y = __shfl_up_sync(kFull, x, o);
+                if (lane >= o) x += y;
+            }
+            if (lane == 31) S.wsum[warp] = x;
+            __syncthreads();
+            unsigned int before = 0;
+            for (int w = 0; w < warp; ++w) before += S.wsum[w];
+            unsigned int run = before + x - t;
+#pragma unroll
+            for (int q = 0; q < 4; ++q) {
+                const unsigned int i = threadIdx.x * 4 + q;
+                if (i < ns) { S.sub[i] = run; S.cur[i] = run; }
+                run += c[q];
+            }
+            if (threadIdx.x == kBkThreads - 1) S.sub[ns] = run;
+        }
+        __syncthreads();
+        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
+            const unsigned long long kk = S.k1[i];
+            const unsigned int p = atomicAdd(&S.cur[(unsigned int)(kk >> ssh) & smask], 1u);
+            S.k2[p] = kk;
+            S.v2[p] = S.v1[i];
+        }
+        __syncthreads();
+        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {  // rank -> sorted smem
+            const unsigned long long kk = S.k2[i], vv = S.v2[i];
+            const unsigned int sbk = (unsigned int)(kk >> ssh) & smask;
+            const unsigned int s0 = S.sub[sbk], s1 = S.sub[sbk + 1];
+            unsigned int rank = s0;
+            for (unsigned int j = s0; j < s1; ++j) {
+                const unsigned long long kj = S.k2[j], vj = S.v2[j];
+                rank += (kj < kk) | ((kj == kk) & ((vj < vv) | ((vj == vv) & (j < i))));
+            }
+            S.k1[rank] = kk;
+            S.v1[rank] = vv;
+        }
+        __syncthreads();
+        const unsigned int cur_lo = lo, cur_m = m;
+        fetch(wi + gridDim.x);  // next bucket's records in flight during the stores below
+        for (unsigned int i = threadIdx.x; i <= ns; i += kBkThreads) S.sub[i] = 0;
+        for (unsigned int i = threadIdx.x; i < cur_m; i += kBkThreads) {  // decode + coalesced stores
+            const CarryRow c = carry_decode(S.k1[i], S.v1[i], sp);
+            const uint64_t j = cur_lo + i;
+            dst.c_last[j] = c.c_last;
+            dst.c_id[j] = c.c_id;
+            dst.o_id[j] = c.o_id;
+            dst.o_entry_d[j] = c.o_entry_d;
+            dst.o_ol_cnt[j] = c.o_ol_cnt;
+            dst.amount_sum[j] = c.amount;
+            dst.o_w_id[j] = c.o_w_id;
+            dst.o_d_id[j] = c.o_d_id;
+        }
+        __syncthreads();
+    }
+}
+
 // 3. One block per bucket: partition by the next `sb` key bits into sub-buckets, rank every row
 // inside its sub-bucket, order equal-prefix runs by the full tuple, and write the result columns
 // at their final positions. The small instance walks every bucket and queues buckets above its
@@ -486,6 +697,11 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
                          const long long *__restrict__ amt, Q18Cols dst, unsigned int *flag,
                          unsigned int *big) {
     extern __shared__ __align__(16) unsigned char smem_raw[];
+    if (kPairs && plan->spec.carry) {  // uniform: the whole ORDER BY runs on carry records
+        carry_sort_emit<(kMin > 0 ? kLcCapLarge : kLsCap), kMin>(
+            reinterpret_cast<const ulonglong2 *>(k), offset, nb, plan, dst, flag, big, smem_raw);
+        return;
+    }
     LsSmem<kLsCap> &S = *reinterpret_cast<LsSmem<kLsCap> *>(smem_raw);
     const int shift = plan->shift;
     const Q18SortSpec sp = plan->spec;
@@ -669,6 +885,11 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
 constexpr int kObThreads = 1024;   // hist / scatter: 2 blocks of 32 warps per SM
 constexpr int kObCap = kLsCapSmall;  // per-bucket sort capacity: 2 048 rows (56 KB, 3 blocks/SM);
                                      // 4 096 (2 blocks/SM) with ~730-row buckets measured slower
+// dynamic shared memory of the v2 emit instances: row-id or carry layout, whichever is larger
+constexpr size_t kObSmem = sizeof(LsSmem<kObCap>) > sizeof(LcSmem<kObCap>) ? sizeof(LsSmem<kObCap>)
+                                                                           : sizeof(LcSmem<kObCap>);
+constexpr size_t kObSmemLarge = sizeof(LsSmem<kLsCapLarge>) > sizeof(LcSmem<kLcCapLarge>)
+                                    ? sizeof(LsSmem<kLsCapLarge>) : sizeof(LcSmem<kLcCapLarge>);
 
 __device__ __forceinline__ unsigned int ob_bucket(const Q18Row *rows, const long long *amt, uint64_t i,
                                                   const Q18SortSpec &sp, int shift, bool amt_only) {
@@ -824,9 +1045,10 @@ ob_scatter_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__
         for (int u = 0; u < U; ++u) {
             const uint64_t i = i0 + (uint64_t)u * kObThreads;
             if (i >= r1) break;
-            const unsigned long long kk = prefix_key(r[u], a[u], sp);
-            const unsigned int p = atomicAdd(&cur[(unsigned int)(kk >> shift)], 1u);
-            reinterpret_cast<ulonglong2 *>(kvout)[p] = make_ulonglong2(kk, (unsigned long long)i);
+            const ulonglong2 rec = sp.carry ? carry_record(r[u], a[u], sp)
+                                            : make_ulonglong2(prefix_key(r[u], a[u], sp), (unsigned long long)i);
+            const unsigned int p = atomicAdd(&cur[(unsigned int)(rec.x >> shift)], 1u);
+            reinterpret_cast<ulonglong2 *>(kvout)[p] = rec;
         }
     }
 }
@@ -906,9 +1128,9 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
     static bool init = false;
     if (!init) {
         cudaFuncSetAttribute(bucket_local_emit_kernel<kObCap, 0, true>,
-                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kObCap>));
+                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kObSmem);
         cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>,
-                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapLarge>));
+                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kObSmemLarge);
         cudaFuncSetAttribute(ob_hist_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 << kBucketMaxBits);
         cudaFuncSetAttribute(ob_scatter_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 << kBucketMaxBits);
         cudaFuncSetAttribute(ob_scan_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
@@ -932,13 +1154,13 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
     // per-bucket shared-memory sort + tie-fix + emit: the v1 kernels on the (key, row id) pairs
     begin("q18_bucket_sort_emit");
     const unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
-    bucket_local_emit_kernel<kObCap, 0, true><<<lb, kBkThreads, sizeof(LsSmem<kObCap>), st>>>(
+    bucket_local_emit_kernel<kObCap, 0, true><<<lb, kBkThreads, kObSmem, st>>>(
         s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
     end();
     begin("q18_bucket_sort_emit_large");
     bucket_local_emit_kernel<kLsCapLarge, kObCap, true><<<(unsigned)num_sms, kBkThreads,
-                                                                sizeof(LsSmem<kLsCapLarge>), st>>>(
+                                                                kObSmemLarge, st>>>(
         s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
     end();

@@ -61,6 +61,17 @@ def L(h, eng):
     return Loader(h, eng)
 
 
+@pytest.fixture(params=["carry", "rowid"])
+def order_mode(request, monkeypatch):
+    """The ORDER BY's two record layouts: 128-bit carry records (default when
+    the row fits) and (64-bit prefix, row id) pairs with tie-fix / exact fallback."""
+    if request.param == "rowid":
+        monkeypatch.setenv("H2TAP_ORDER_CARRY", "0")
+    else:
+        monkeypatch.delenv("H2TAP_ORDER_CARRY", raising=False)
+    return request.param
+
+
 def assert_q6(got, want):
     assert got["count_rows"][0] == want["count"]
     if want["revenue"] is None:
@@ -129,7 +140,7 @@ def test_golden_fixture(L):
 
 
 @pytest.mark.parametrize("W,mode,seed", [(1, "spread", 1), (3, "spread", 2), (2, "strict", 3)])
-def test_parity_small(L, W, mode, seed):
+def test_parity_small(L, W, mode, seed, order_mode):
     run_all(L, chgen.generate(1, W + 1, seed=seed, mode=mode), np.random.default_rng(seed))
 
 
@@ -178,7 +189,7 @@ def test_q6_quantity_and_null_edges(L):
         assert_q6(L.q(6, p), oracle.q6(t, *p))
 
 
-def test_q18_join_edges(L):
+def test_q18_join_edges(L, order_mode):
     """Orphan lines, orders without lines, customers missing, negative HAVING."""
     t = chgen.generate(1, 2, seed=6)
     ol, o, c = t["order_line"], t["orders"], t["customer"]
@@ -195,7 +206,7 @@ def test_q18_join_edges(L):
         assert_q18(L.q(18, [thr], flags=HASH), want)
 
 
-def test_q18_ties_use_full_order(L):
+def test_q18_ties_use_full_order(L, order_mode):
     """Equal amount_sum and o_entry_d: the (w, d, o) tie-break decides (R11)."""
     t = chgen.generate(1, 3, seed=9)
     t["order_line"]["ol_amount"][:] = 1000
@@ -205,7 +216,7 @@ def test_q18_ties_use_full_order(L):
         assert_q18(L.q(18, [thr]), oracle.q18(t, thr))
 
 
-def test_q18_sort_fallback_long_prefix_runs(L):
+def test_q18_sort_fallback_long_prefix_runs(L, order_mode):
     """Composite key > 64 bits and > 32 rows sharing the 48-bit prefix: exact field-by-field
     re-sort path."""
     for variant in ("short_runs", "long_runs"):
@@ -222,6 +233,39 @@ def test_q18_sort_fallback_long_prefix_runs(L):
             want = oracle.q18(t, thr)
             assert_q18(L.q(18, [thr]), want)
             assert_q18(L.q(18, [thr], flags=HASH), want)
+
+
+def test_q18_wide_payload_disables_carry(L):
+    """c_last codes spanning 32 bits (and a 96-bit key): the carry record cannot hold the row,
+    the plan falls back to row-id pairs on its own (no env knob)."""
+    t = chgen.generate(1, 3, seed=23)
+    rng = np.random.default_rng(23)
+    c = t["customer"]
+    c["c_last"][:] = rng.integers(-2**31, 2**31 - 1, len(c["c_last"]), dtype=np.int64).astype(np.int32)
+    L.load(t)
+    for thr in (0, Q18_HAVING):
+        want = oracle.q18(t, thr)
+        assert_q18(L.q(18, [thr]), want)
+        assert_q18(L.q(18, [thr], flags=HASH), want)
+
+
+def test_q18_carry_field_extremes(L):
+    """Carry decode with full 128-bit records: 44-bit amount_sum field, o_entry_d far below 1970
+    (negative µs), a 17-bit o_ol_cnt payload field; a negative o_ol_cnt (32-bit field) no
+    longer fits and the plan falls back to row ids."""
+    t = chgen.generate(1, 2, seed=29)
+    o, c = t["orders"], t["customer"]
+    o["o_entry_d"][:] = -(10**15) + np.arange(len(o["o_id"]), dtype=np.int64) * 7919
+    o["o_ol_cnt"][::3] = 1 << 16                  # 17-bit o_ol_cnt field, record still fits
+    t["order_line"]["ol_amount"][::5] = 10**12
+    L.load(t)
+    for thr in (-10**13, 0, 10**12):
+        want = oracle.q18(t, thr)
+        assert_q18(L.q(18, [thr]), want)
+    o["o_ol_cnt"][::7] = -5
+    L.load(t)
+    for thr in (0, 10**12):
+        assert_q18(L.q(18, [thr]), oracle.q18(t, thr))
 
 
 def test_q18_planner_dense_and_hash(h, eng, L):
