@@ -14,6 +14,7 @@
 //    per-digit scan -> stable scatter; keys travel with their row ids.
 #include <algorithm>
 #include <cstdint>
+#include <cstdlib>
 #include <cuda_runtime.h>
 
 #include "cache_hints.cuh"
@@ -558,7 +559,8 @@ template <int kCap, int kMin>
 __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ kv,
                                                 const unsigned int *__restrict__ offset, int nb,
                                                 const Q18Plan *__restrict__ plan, const Q18Cols &dst,
-                                                unsigned int *flag, unsigned int *big, unsigned char *smem) {
+                                                unsigned int *flag, unsigned int *big, unsigned char *smem,
+                                                int sub_log2) {
     LcSmem<kCap> &S = *reinterpret_cast<LcSmem<kCap> *>(smem);
     const int shift = plan->shift;
     const Q18SortSpec sp = plan->spec;
@@ -597,7 +599,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
             continue;
         }
         int sb = 0;
-        while (sb < 10 && (m >> (sb + 3)) > 0) ++sb;
+        while (sb < 10 && (m >> (sb + sub_log2)) > 0) ++sb;
         if (sb > shift) sb = shift;
         const int ssh = shift - sb;
         const unsigned int ns = 1u << sb, smask = ns - 1u;
@@ -690,16 +692,16 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
 // capacity in big[1..]; the large instance walks only that queue.
 // kPairs: k holds interleaved 16-byte (key, row id) pairs (v2 scatter), v is unused.
 template <int kLsCap, int kMin, bool kPairs = false>
-__global__ void __launch_bounds__(kBkThreads)
+__global__ void __launch_bounds__(kBkThreads, 3)
 bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigned int *__restrict__ v,
                          const unsigned int *__restrict__ offset, int nb,
                          const Q18Plan *__restrict__ plan, const Q18Row *__restrict__ rows,
                          const long long *__restrict__ amt, Q18Cols dst, unsigned int *flag,
-                         unsigned int *big) {
+                         unsigned int *big, int sub_log2 = 3) {
     extern __shared__ __align__(16) unsigned char smem_raw[];
     if (kPairs && plan->spec.carry) {  // uniform: the whole ORDER BY runs on carry records
         carry_sort_emit<(kMin > 0 ? kLcCapLarge : kLsCap), kMin>(
-            reinterpret_cast<const ulonglong2 *>(k), offset, nb, plan, dst, flag, big, smem_raw);
+            reinterpret_cast<const ulonglong2 *>(k), offset, nb, plan, dst, flag, big, smem_raw, sub_log2);
         return;
     }
     LsSmem<kLsCap> &S = *reinterpret_cast<LsSmem<kLsCap> *>(smem_raw);
@@ -1138,6 +1140,11 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
         init = true;
     }
     (void)n_max;
+    // carry sort: ~2^sub_log2 rows per sub-bucket (rank loop vs sub-bucket scan; knob for A/B)
+    static const int sub_log2 = [] {
+        const char *v = std::getenv("H2TAP_SUB_ROWS_LOG2");
+        return v ? std::max(0, std::min(6, std::atoi(v))) : 1;  // measured: 1 -> 74 us, 3 -> 84 us
+    }();
     begin("q18_sort_hist");
     ob_hist_kernel<<<G, kObThreads, nb * 4, st>>>(rows, amt, plan, nb, s.mat, s.big);
     count_launches(1);
@@ -1155,13 +1162,13 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
     begin("q18_bucket_sort_emit");
     const unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
     bucket_local_emit_kernel<kObCap, 0, true><<<lb, kBkThreads, kObSmem, st>>>(
-        s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big);
+        s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2);
     count_launches(1);
     end();
     begin("q18_bucket_sort_emit_large");
     bucket_local_emit_kernel<kLsCapLarge, kObCap, true><<<(unsigned)num_sms, kBkThreads,
                                                                 kObSmemLarge, st>>>(
-        s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big);
+        s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2);
     count_launches(1);
     end();
 }
