@@ -342,11 +342,30 @@ def main():
             _ = r.columns[next(iter(r.columns))][:1].sum() if r.nrows else 0  # host read
             h.h2tap_free(r)
     barrier()
-    e2e_s = (time.perf_counter() - t0) / e2e_steps
-    te = torch.tensor([e2e_s], dtype=torch.float64, device="cuda")
+    e2e_serial_s = (time.perf_counter() - t0) / e2e_steps
+    # pipelined: the same calls with H2TAP_LOAD_ASYNC | H2TAP_LOAD_BORROW (the pinned buffers are
+    # lent to the DMA and not modified), so step k's 1.2 GB upload (copy stream)
+    # overlaps step k-1's result read-back (D2H, the other PCIe direction) and the queries; each
+    # batch runs on the latest PUBLISHED epoch (k or k-1, reported per step) — double buffering
+    h.h2tap_sync(eng)
+    barrier()
+    lag = []
+    t0 = time.perf_counter()
+    for _ in range(e2e_steps):
+        epoch += 1
+        h.h2tap_load_snapshot(eng, pinned, epoch, flags=h.H2TAP_LOAD_ASYNC | h.H2TAP_LOAD_BORROW)
+        for r in h.h2tap_run_queries(eng, [(plan, p, 0) for _, plan, p in plans]):
+            _ = r.columns[next(iter(r.columns))][:1].sum() if r.nrows else 0  # host read
+            lag.append(epoch - r.epoch)
+            h.h2tap_free(r)
+    h.h2tap_sync(eng)  # the last upload is inside the timed region too
+    barrier()
+    e2e_pipe_s = (time.perf_counter() - t0) / e2e_steps
+    te = torch.tensor([e2e_serial_s, e2e_pipe_s], dtype=torch.float64, device="cuda")
     if world > 1:
         dist.all_reduce(te, op=dist.ReduceOp.MAX)
-    e2e_s = float(te.item())
+    e2e_serial_s, e2e_pipe_s = (float(x) for x in te.tolist())
+    e2e_s = min(e2e_serial_s, e2e_pipe_s)
 
     # ---- CPU oracle baseline (rank 0, N = 1 only, bounded sample)
     cpu = None
@@ -376,7 +395,15 @@ def main():
             "kernels": kernels_summary,
             "cpu_baseline": cpu,
             "e2e": {"value": rows_total / e2e_s, "unit": UNIT, "h2d_bytes_per_step": int(h2d_bytes),
-                    "d2h_bytes_per_step": int(d2h), "ms_per_step": e2e_s * 1e3, "steps": e2e_steps},
+                    "d2h_bytes_per_step": int(d2h), "ms_per_step": e2e_s * 1e3, "steps": e2e_steps,
+                    "mode": "pipelined" if e2e_pipe_s <= e2e_serial_s else "serial",
+                    "serial_ms_per_step": e2e_serial_s * 1e3, "pipelined_ms_per_step": e2e_pipe_s * 1e3,
+                    "pipelined_epoch_lag": sorted(set(lag)),
+                    "how": "every step: full snapshot upload of the step's inputs from pinned host "
+                           "buffers (h2tap_load_snapshot) + Q6/Q1/Q18 batch (h2tap_run_queries) + "
+                           "results copied to host; serial = load then queries; pipelined = "
+                           "H2TAP_LOAD_ASYNC|H2TAP_LOAD_BORROW, queries on the latest published "
+                           "epoch (lag in epochs listed)"},
             "gpu_launches": int(launches),
             "clocks": clk,
         }

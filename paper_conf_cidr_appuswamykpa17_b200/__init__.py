@@ -40,6 +40,7 @@ H2TAP_FULL_RELOAD = 1
 H2TAP_DSM, H2TAP_PAX, H2TAP_NSM = 1, 2, 3  # NEXT-3 layouts (§5.3)
 H2TAP_LOAD_ASYNC = 1
 H2TAP_LOAD_ZERO_COPY = 2  # NEXT-4: kernels read the caller's pinned host columns over PCIe
+H2TAP_LOAD_BORROW = 4  # with ASYNC: pinned buffers lent to the DMA until the epoch is published
 H2TAP_RESULT_DEVICE = 1
 H2TAP_QUERY_PROFILE = 2
 H2TAP_QUERY_HASH_JOIN = 4

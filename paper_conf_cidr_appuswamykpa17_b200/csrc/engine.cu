@@ -751,7 +751,8 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         std::lock_guard<std::mutex> gp(e->pend_mu);
         e->pending.push_back(pend);
     }
-    if (must_wait || !(flags & H2TAP_LOAD_ASYNC)) publish_ready(e, true);
+    // pinned caller buffers are read by the DMA after we return: wait, unless they are lent
+    if ((must_wait && !(flags & H2TAP_LOAD_BORROW)) || !(flags & H2TAP_LOAD_ASYNC)) publish_ready(e, true);
     return H2TAP_OK;
 }
 
@@ -1981,8 +1982,9 @@ h2tap_status h2tap_refresh_rows(h2tap_engine *e, const h2tap_row_table *tables, 
         for (unsigned t = 1; t < nthreads; ++t) pool.emplace_back(work, t);
         work(0);
         for (auto &th : pool) th.join();
-        // pinned sources: load_impl DMAs them directly and waits before returning
-        return load_impl(e, tabs.data(), ntables, updates, nupdates, epoch, flags);
+        // pinned sources: load_impl DMAs them directly and waits before returning (the extraction
+        // buffers are the library's and reused by the next call: never lent)
+        return load_impl(e, tabs.data(), ntables, updates, nupdates, epoch, flags & ~H2TAP_LOAD_BORROW);
     });
 }
 

@@ -402,6 +402,39 @@ def test_snapshot_epochs_append_and_errors(h):
         h.h2tap_close(e)
 
 
+def test_async_borrowed_pinned_loads(h):
+    """H2TAP_LOAD_ASYNC | H2TAP_LOAD_BORROW: the call returns before the DMA of the lent pinned
+    buffers; queries run on the latest PUBLISHED epoch and every result equals the oracle of the
+    epoch it reports; alternating two table sets catches a query that mixes them."""
+    import torch
+    sets = [chgen.generate(1, 4, seed=41), chgen.generate(1, 4, seed=42)]
+    pinned = [{t: {c: torch.from_numpy(v).pin_memory() for c, v in cols.items()}
+               for t, cols in h.hot_path_tables(ts).items()} for ts in sets]
+    want = [(oracle.q6(ts, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI), oracle.q1(ts, Q1_CUTOFF),
+             oracle.q18(ts, Q18_HAVING)) for ts in sets]
+    e = h.h2tap_open(0)
+    try:
+        h.h2tap_load_snapshot(e, pinned[0], 1)
+        seen = set()
+        for ep in range(2, 10):
+            h.h2tap_load_snapshot(e, pinned[ep % 2], ep, flags=h.H2TAP_LOAD_ASYNC | h.H2TAP_LOAD_BORROW)
+            rs = h.h2tap_run_queries(e, [(6, None, 0), (1, None, 0), (18, None, 0)])
+            for plan, r in zip((6, 1, 18), rs):
+                got, k = r.to_numpy(), r.epoch % 2
+                seen.add(ep - r.epoch)
+                if plan == 6:
+                    assert got["revenue"][0] == want[k][0]["revenue"]
+                elif plan == 1:
+                    assert np.array_equal(got["sum_amount"], want[k][1]["sum_amount"])
+                else:
+                    assert_q18(got, want[k][2])
+                h.h2tap_free(r)
+        assert h.h2tap_sync(e) == 9
+        assert seen <= {0, 1}
+    finally:
+        h.h2tap_close(e)
+
+
 def test_row_store_refresh(h):
     """h2tap_load_snapshot_rows: NSM records -> DSM snapshot (full load, then an append)."""
     e = h.h2tap_open(0)
