@@ -138,8 +138,11 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes):
         "q18_sort_keys_hist": (32 + 8 + 8 + 4) * n_pass,   # rows + amounts -> keys + row ids
         # ORDER BY v2 (default): count matrix + scatter computing keys + chunked local sort
         "q18_sort_hist": 8 * n_pass,                       # amounts (bucket bits inside field a)
-        "q18_bucket_scatter": (40 + 16) * n_pass if sort_passes == "v2" else (12 + 12) * n_pass,
-        "q18_bucket_sort_emit": (16 if sort_passes == "v2" else 12) * n_pass + (32 + 40) * n_pass,
+        "q18_bucket_scatter": (40 + 16) * n_pass if sort_passes != "v1" else (12 + 12) * n_pass,
+        # carry records (v2 default): 16 B record in, 40 B of result columns out (no row gather);
+        # row-id paths: pair in + 32 B row gather + 40 B out
+        "q18_bucket_sort_emit": (16 + 40) * n_pass if sort_passes == "carry"
+                                else (16 if sort_passes == "v2" else 12) * n_pass + (32 + 40) * n_pass,
     }.get(kernel)
 
 
@@ -300,7 +303,8 @@ def main():
 
     # ---- roofline for the dominant kernel (largest share of the step)
     kavg = {k: float(np.mean(v)) for k, v in kern.items()}
-    sort_passes = "v1" if os.environ.get("H2TAP_ORDER") == "v1" else "v2"
+    sort_passes = ("v1" if os.environ.get("H2TAP_ORDER") == "v1"
+                   else "v2" if os.environ.get("H2TAP_ORDER_CARRY") == "0" else "carry")
     dominant = max(kavg, key=kavg.get) if kavg else None
     peak, peak_src = peaks()
     roof = None
