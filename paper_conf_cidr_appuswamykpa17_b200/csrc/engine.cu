@@ -34,6 +34,10 @@
 namespace h2tap {
 static std::atomic<uint64_t> g_launches{0};
 void count_launches(int n) { g_launches.fetch_add((uint64_t)n, std::memory_order_relaxed); }
+bool pdl_enabled() {
+    static const bool on = [] { const char *v = std::getenv("H2TAP_PDL"); return !(v && v[0] == '0'); }();
+    return on;
+}
 uint64_t launches_total() { return g_launches.load(std::memory_order_relaxed); }
 }  // namespace h2tap
 

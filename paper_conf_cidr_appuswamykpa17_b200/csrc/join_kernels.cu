@@ -38,6 +38,8 @@ unsigned grid_for(uint64_t work, int threads, int num_sms, int per_sm) {
 // Empties both join indexes, zeroes the group accumulators and the counters: one launch.
 // Empties both join indexes, zeroes the group accumulators and the counters: one launch.
 __global__ void q18_init_kernel(Q18Scratch s) {
+    pdl_wait();
+    pdl_trigger();
     const uint64_t a = jx_words(s.jo), b = jx_words(s.jc), q = s.qbits ? s.qwords : 0;
     const uint64_t total = a + b + q;  // (the accumulators are zeroed by the build, row by row)
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
@@ -62,6 +64,8 @@ __global__ void q18_build_kernel(const int32_t *__restrict__ o_w, const int32_t 
                                  const int32_t *__restrict__ o_id, uint64_t n_o,
                                  const int32_t *__restrict__ c_w, const int32_t *__restrict__ c_d,
                                  const int32_t *__restrict__ c_id, uint64_t n_c, Q18Scratch s) {
+    pdl_wait();
+    pdl_trigger();
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n_o + n_c; i += stride) {
         bool ok;
@@ -168,6 +172,8 @@ __global__ void __launch_bounds__(kProbeThreads)
 q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ ol_d,
                  const int32_t *__restrict__ ol_o, const int64_t *__restrict__ ol_amt, uint64_t n,
                  Q18Scratch s) {
+    pdl_wait();
+    pdl_trigger();
     const int lane = threadIdx.x & 31;
     const uint64_t gwarp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
@@ -370,6 +376,8 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
                   const int32_t *__restrict__ o_id, const int32_t *__restrict__ o_c,
                   const int32_t *__restrict__ o_cnt, const int64_t *__restrict__ o_ent, uint64_t n,
                   const int32_t *__restrict__ c_last, long long having, Q18Scratch s) {
+    pdl_wait();
+    pdl_trigger();
     __shared__ unsigned int wsum[kHavingThreads / 32];
     __shared__ unsigned long long s_base;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -569,6 +577,8 @@ q3_emit_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
 struct Q18SmallDev { unsigned long long nout; unsigned int err, tie; };  // = engine's Q18Small head
 __global__ void q18_publish_kernel(const unsigned long long *nout, const unsigned int *err,
                                    const unsigned int *tie, Q18SmallDev *out) {
+    pdl_wait();
+    pdl_trigger();
     out->nout = *nout;
     out->err = *err;
     out->tie = *tie;
@@ -578,21 +588,21 @@ __global__ void q18_publish_kernel(const unsigned long long *nout, const unsigne
 
 void launch_q18_publish(const unsigned long long *nout, const unsigned int *err, const unsigned int *tie,
                         void *host_small, cudaStream_t st) {
-    q18_publish_kernel<<<1, 1, 0, st>>>(nout, err, tie, static_cast<Q18SmallDev *>(host_small));
+    launch_pdl(q18_publish_kernel, 1, 1, 0, st, nout, err, tie, static_cast<Q18SmallDev *>(host_small));
     count_launches(1);
 }
 
 void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st) {
     (void)n_orders;
     const uint64_t words = jx_words(s.jo) + jx_words(s.jc);
-    q18_init_kernel<<<grid_for(words, 256, num_sms, 8), 256, 0, st>>>(s);
+    launch_pdl(q18_init_kernel, grid_for(words, 256, num_sms, 8), 256, 0, st, s);
     count_launches(1);
 }
 
 void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
                       const int32_t *c_w, const int32_t *c_d, const int32_t *c_id, uint64_t n_c,
                       const Q18Scratch &s, int num_sms, cudaStream_t st) {
-    q18_build_kernel<<<grid_for(n_o + n_c, 256, num_sms, 8), 256, 0, st>>>(o_w, o_d, o_id, n_o, c_w,
+    launch_pdl(q18_build_kernel, grid_for(n_o + n_c, 256, num_sms, 8), 256, 0, st, o_w, o_d, o_id, n_o, c_w,
                                                                          c_d, c_id, n_c, s);
     count_launches(1);
 }
@@ -600,7 +610,7 @@ void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_i
 void launch_q18_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
                       const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
                       cudaStream_t st) {
-    q18_probe_kernel<false><<<grid_for((n_ol + 3) / 4, kProbeThreads, num_sms, 8), kProbeThreads, 0, st>>>(
+    launch_pdl(q18_probe_kernel<false>, grid_for((n_ol + 3) / 4, kProbeThreads, num_sms, 8), kProbeThreads, 0, st,
         ol_w, ol_d, ol_o, ol_amt, n_ol, s);
     count_launches(1);
 }
@@ -657,10 +667,10 @@ void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_
         return v ? std::max(1, std::min(8, std::atoi(v))) : 4;
     }();
     if (unroll == 4)
-        q18_having_kernel<4><<<grid_for((n_o + 3) / 4, kHavingThreads, num_sms, bps), kHavingThreads, 0, st>>>(
+        launch_pdl(q18_having_kernel<4>, grid_for((n_o + 3) / 4, kHavingThreads, num_sms, bps), kHavingThreads, 0, st,
             o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o, c_last, having, s);
     else
-        q18_having_kernel<2><<<grid_for((n_o + 1) / 2, kHavingThreads, num_sms, bps), kHavingThreads, 0, st>>>(
+        launch_pdl(q18_having_kernel<2>, grid_for((n_o + 1) / 2, kHavingThreads, num_sms, bps), kHavingThreads, 0, st,
             o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o, c_last, having, s);
     count_launches(1);
 }

@@ -3,6 +3,7 @@
 #pragma once
 #include <cstdint>
 #include <cuda_runtime.h>
+#include <utility>
 
 namespace h2tap {
 
@@ -251,6 +252,30 @@ void launch_apply_updates(void *col, uint32_t es, uint32_t *bits, const uint32_t
 // ---------------------------------------------------------------- helpers --
 // Every launcher counts the kernels it launches (reported per query as kernel_launches).
 void count_launches(int n);
+
+// Programmatic dependent launch: the hot-path kernels of a batch are launched
+// with programmatic stream serialization, so kernel k+1 is already resident when kernel k ends
+// (launch latency and its block scheduling overlap k's tail). Every such kernel starts with
+// pdl_wait() — it returns once the preceding grid has completed and its writes are visible — and
+// pdl_trigger(), which lets the next grid launch. H2TAP_PDL=0 launches them normally (A/B).
+__device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+__device__ __forceinline__ void pdl_trigger() { asm volatile("griddepcontrol.launch_dependents;" ::: "memory"); }
+bool pdl_enabled();
+template <typename... KArgs, typename... Args>
+inline void launch_pdl(void (*kern)(KArgs...), dim3 grid, dim3 block, size_t smem, cudaStream_t st,
+                       Args &&...args) {
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    at[0].val.programmaticStreamSerializationAllowed = pdl_enabled() ? 1 : 0;
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = grid;
+    cfg.blockDim = block;
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = st;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    cudaLaunchKernelEx(&cfg, kern, std::forward<Args>(args)...);
+}
 
 // ------------------------------------------- NEXT-2: CH Q14 / Q12 / Q4 (ch_kernels.cu) --
 // GROUP BY o_ol_cnt with counters (a, b, rows) per group: keys in [0, kSgDense) in thread-private

@@ -172,6 +172,8 @@ q6_tma_kernel(const long long *__restrict__ deliv, const int *__restrict__ qty,
               const long long *__restrict__ amt, uint64_t n, Q6Pred pred,
               long long *__restrict__ part, unsigned int *__restrict__ counter,
               long long *__restrict__ out, long long *__restrict__ host_out) {
+    pdl_wait();
+    pdl_trigger();
     extern __shared__ __align__(128) unsigned char smem_raw[];
     Q6TmaSmem &S = *reinterpret_cast<Q6TmaSmem *>(smem_raw);
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
@@ -469,6 +471,8 @@ __global__ void __launch_bounds__(kTmaThreads, 1)
 q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deliv,
               const int *__restrict__ qty, const long long *__restrict__ amt, uint64_t n,
               long long cutoff, Q1Scratch g) {
+    pdl_wait();
+    pdl_trigger();
     extern __shared__ __align__(128) unsigned char smem_raw[];
     Q1Stages &P = *reinterpret_cast<Q1Stages *>(smem_raw);
     Q1Smem &sm = *reinterpret_cast<Q1Smem *>(smem_raw + sizeof(Q1Stages));
@@ -543,6 +547,8 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
 
 // Collect the dense and global tables into groups[] and clear them for the next query.
 __global__ void q1_compact_kernel(Q1Scratch g) {
+    pdl_wait();
+    pdl_trigger();
     const uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
     if (i < (uint64_t)kQ1Dense) {
         const unsigned long long c = g.dense[3 * i];
@@ -579,6 +585,8 @@ __global__ void q1_merge_kernel(const Q1Group *__restrict__ all, uint64_t n, Q1S
 // ORDER BY ol_number: keys are distinct, so each group's output position is its rank
 // (number of smaller keys). AVG = SUM / COUNT in IEEE double, money / 100 (R7).
 __global__ void q1_emit_kernel(Q1Scratch g) {
+    pdl_wait();
+    pdl_trigger();
     __shared__ long long tile[1024];
     const uint64_t ng = *g.ngroups;  // read on the device: no host round trip before emitting
     if (g.host_small && blockIdx.x == 0 && threadIdx.x == 0) {  // mapped pinned: no D2H copies
@@ -640,7 +648,7 @@ void launch_q6_tma(const int64_t *deliv, const int32_t *qty, const int64_t *amt,
     }
     const uint64_t nchunks = (n + kQ6Chunk - 1) / kQ6Chunk;
     const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
-    q6_tma_kernel<<<grid, kTmaThreads, sizeof(Q6TmaSmem), st>>>(
+    launch_pdl(q6_tma_kernel, grid, kTmaThreads, sizeof(Q6TmaSmem), st,
         reinterpret_cast<const long long *>(deliv), qty, reinterpret_cast<const long long *>(amt), n,
         Q6Pred{d_lo, d_hi, q_lo, q_hi}, s.block_part, s.done_counter, s.out, s.host_out);
     count_launches(1);
@@ -684,13 +692,13 @@ void launch_q1_tma(const int32_t *number, const int64_t *deliv, const int32_t *q
     }
     const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
     const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
-    q1_tma_kernel<<<grid, kTmaThreads, smem, st>>>(number, reinterpret_cast<const long long *>(deliv), qty,
+    launch_pdl(q1_tma_kernel, grid, kTmaThreads, smem, st, number, reinterpret_cast<const long long *>(deliv), qty,
                                                    reinterpret_cast<const long long *>(amt), n, cutoff, s);
     count_launches(1);
 }
 
 void launch_q1_compact(const Q1Scratch &s, cudaStream_t st) {
-    q1_compact_kernel<<<kQ1GlobalSlots / 256, 256, 0, st>>>(s);
+    launch_pdl(q1_compact_kernel, kQ1GlobalSlots / 256, 256, 0, st, s);
     count_launches(1);
 }
 
@@ -700,7 +708,7 @@ void launch_q1_merge(const Q1Group *all, uint64_t n, const Q1Scratch &s, cudaStr
 }
 
 void launch_q1_emit(const Q1Scratch &s, uint64_t max_groups, cudaStream_t st) {
-    q1_emit_kernel<<<(unsigned)((max_groups + 255) / 256), 256, 0, st>>>(s);
+    launch_pdl(q1_emit_kernel, (unsigned)((max_groups + 255) / 256), 256, 0, st, s);
     count_launches(1);
 }
 

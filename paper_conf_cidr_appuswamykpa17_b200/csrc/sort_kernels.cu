@@ -316,6 +316,8 @@ __device__ __forceinline__ int bitwidth_dev(unsigned long long x) { return x ? 6
 __global__ void q18_plan_kernel(const Q18Stats *__restrict__ stats, Q18Zone z,
                                 const unsigned long long *nout, int bucket_bits, int allow_carry,
                                 Q18Plan *plan, unsigned int *flag) {
+    pdl_wait();
+    pdl_trigger();
     const Q18Stats st = *stats;
     Q18Plan p{};
     p.n = *nout;
@@ -359,7 +361,7 @@ unsigned grid_cap(uint64_t work, int threads, int num_sms, int per_sm) {
 void launch_q18_plan(const Q18Stats *stats, const Q18Zone &zone, const unsigned long long *nout,
                      int bucket_bits, bool allow_carry, Q18Plan *plan, unsigned int *flag,
                      cudaStream_t st) {
-    q18_plan_kernel<<<1, 1, 0, st>>>(stats, zone, nout, bucket_bits, allow_carry ? 1 : 0, plan, flag);
+    launch_pdl(q18_plan_kernel, 1, 1, 0, st, stats, zone, nout, bucket_bits, allow_carry ? 1 : 0, plan, flag);
     count_launches(1);
 }
 
@@ -698,6 +700,8 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
                          const Q18Plan *__restrict__ plan, const Q18Row *__restrict__ rows,
                          const long long *__restrict__ amt, Q18Cols dst, unsigned int *flag,
                          unsigned int *big, int sub_log2 = 3) {
+    pdl_wait();
+    pdl_trigger();
     extern __shared__ __align__(16) unsigned char smem_raw[];
     if (kPairs && plan->spec.carry) {  // uniform: the whole ORDER BY runs on carry records
         carry_sort_emit<(kMin > 0 ? kLcCapLarge : kLsCap), kMin>(
@@ -913,6 +917,8 @@ __global__ void __launch_bounds__(kObThreads)
 ob_hist_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
                const Q18Plan *__restrict__ plan, int nb, unsigned int *__restrict__ mat,
                unsigned int *__restrict__ big) {
+    pdl_wait();
+    pdl_trigger();
     extern __shared__ unsigned int h[];
     if (blockIdx.x == 0 && threadIdx.x == 0) *big = 0;  // work-list count of the emit kernels
     const uint64_t n = plan->n;
@@ -947,6 +953,8 @@ constexpr int kScanWarps = 8;
 __global__ void __launch_bounds__(32 * kScanWarps)
 ob_scan_kernel(unsigned int *__restrict__ mat, int G, int nb, unsigned int *__restrict__ count,
                unsigned int *__restrict__ offset, unsigned int *ticket) {
+    pdl_wait();
+    pdl_trigger();
     extern __shared__ unsigned int tile[];  // [G][32]; the last block reuses it for nb totals
     __shared__ bool last;
     __shared__ unsigned int tot[kScanWarps][32];
@@ -1019,6 +1027,8 @@ __global__ void __launch_bounds__(kObThreads)
 ob_scatter_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
                   const Q18Plan *__restrict__ plan, int nb, const unsigned int *__restrict__ mat,
                   const unsigned int *__restrict__ offset, unsigned long long *__restrict__ kvout) {
+    pdl_wait();
+    pdl_trigger();
     extern __shared__ unsigned int cur[];
     const uint64_t n = plan->n;
     const Q18SortSpec sp = plan->spec;
@@ -1146,28 +1156,27 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
         return v ? std::max(0, std::min(6, std::atoi(v))) : 1;  // measured: 1 -> 74 us, 3 -> 84 us
     }();
     begin("q18_sort_hist");
-    ob_hist_kernel<<<G, kObThreads, nb * 4, st>>>(rows, amt, plan, nb, s.mat, s.big);
+    launch_pdl(ob_hist_kernel, G, kObThreads, nb * 4, st, rows, amt, plan, nb, s.mat, s.big);
     count_launches(1);
     end();
     begin("q18_sort_scan");
-    ob_scan_kernel<<<(nb + 31) / 32, 32 * kScanWarps, 4 * std::max(32 * G, nb), st>>>(s.mat, G, nb, s.count,
+    launch_pdl(ob_scan_kernel, (nb + 31) / 32, 32 * kScanWarps, 4 * std::max(32 * G, nb), st, s.mat, G, nb, s.count,
                                                                                    s.offset, s.ticket);
     count_launches(1);
     end();
     begin("q18_bucket_scatter");
-    ob_scatter_kernel<<<G, kObThreads, nb * 4, st>>>(rows, amt, plan, nb, s.mat, s.offset, s.kv);
+    launch_pdl(ob_scatter_kernel, G, kObThreads, nb * 4, st, rows, amt, plan, nb, s.mat, s.offset, s.kv);
     count_launches(1);
     end();
     // per-bucket shared-memory sort + tie-fix + emit: the v1 kernels on the (key, row id) pairs
     begin("q18_bucket_sort_emit");
     const unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
-    bucket_local_emit_kernel<kObCap, 0, true><<<lb, kBkThreads, kObSmem, st>>>(
+    launch_pdl(bucket_local_emit_kernel<kObCap, 0, true>, lb, kBkThreads, kObSmem, st,
         s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2);
     count_launches(1);
     end();
     begin("q18_bucket_sort_emit_large");
-    bucket_local_emit_kernel<kLsCapLarge, kObCap, true><<<(unsigned)num_sms, kBkThreads,
-                                                                kObSmemLarge, st>>>(
+    launch_pdl(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>, (unsigned)num_sms, kBkThreads, kObSmemLarge, st,
         s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2);
     count_launches(1);
     end();

@@ -1,7 +1,7 @@
-# Q18 ORDER BY iteration: Q18 parity tests, then the bench (default, carry off, register scatter)
+# Q18 iteration: Q18 parity tests, then the bench
 mkdir -p gpurun_out
-timeout 600 python -m pytest tests/test_gpu_parity.py tests/test_gpu_q3.py -q -x --timeout 300 2>&1 | tail -3 | tee gpurun_out/pytest_q18.txt
-for v in default H2TAP_ORDER_CARRY=0 H2TAP_SCATTER=ldg; do
+timeout 600 python -m pytest tests/test_gpu_parity.py tests/test_gpu_q3.py tests/test_gpu_next2.py -q -x --timeout 300 2>&1 | tail -3 | tee gpurun_out/pytest_q18.txt
+for v in default; do
   env $([ $v = default ] || echo $v) timeout 300 python bench.py --no-cpu-baseline --steps 10 2>&1 | tail -1 > gpurun_out/ab_q18.json
   python -c "
 import json; d=json.load(open('gpurun_out/ab_q18.json'))
