@@ -1122,7 +1122,13 @@ void q18_bucket_order(const Q18Row *rows, const long long *amt, const Q18Plan *p
 
 namespace h2tap {
 
-int ob_grid(int num_sms) { return 2 * num_sms; }  // row partitions of the v2 ORDER BY front
+int ob_grid(int num_sms) {  // row partitions of the v2 ORDER BY front (H2TAP_OB_PER_SM, 1..2)
+    static const int per = [] {
+        const char *v = std::getenv("H2TAP_OB_PER_SM");
+        return v ? std::max(1, std::min(2, std::atoi(v))) : 2;
+    }();
+    return per * num_sms;
+}
 int ob_bucket_bits(uint64_t n_max) {  // ~256-512 rows per bucket
     int bb = 1;
     while (bb < kBucketMaxBits && (n_max >> (bb + 9)) > 0) ++bb;
