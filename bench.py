@@ -123,17 +123,35 @@ def ncu_traffic():
 
 
 # ------------------------------------------------------------- algorithmic bytes --
-def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes):
-    """Bytes the method must move per launch."""
-    cap_o = 1 << max(4, int(np.ceil(np.log2(max(2 * n_o, 16)))))
-    cap_c = 1 << max(4, int(np.ceil(np.log2(max(2 * n_c, 16)))))
+def key_box(t, cols):
+    """Slots of the (w, d, id) min/max box: the perfect-hash join index size."""
+    n = 1
+    for c in cols:
+        v = t[c]
+        n *= int(v.max()) - int(v.min()) + 1 if len(v) else 0
+    return n
+
+
+def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None):
+    """Bytes the method must move per launch. `box`: the
+    (orders, customer) key-box slot counts when the planner chose perfect-hash indexes (4-byte
+    slots), else None (open addressing: 16-byte slots, capacity pow2 >= 2n)."""
+    if box:
+        slots_o, slots_c, slot_b = box[0], box[1], 4
+    else:
+        slots_o = 1 << max(4, int(np.ceil(np.log2(max(2 * n_o, 16)))))
+        slots_c = 1 << max(4, int(np.ceil(np.log2(max(2 * n_c, 16)))))
+        slot_b = 16
     return {
         "q6_scan_filter_sum": 20 * n_ol,
         "q1_scan_filter_groupby": 24 * n_ol,
-        "q18_init": 16 * (cap_o + cap_c + n_o),
-        "q18_build": 12 * n_o + 12 * n_c + 16 * (n_o + n_c),
-        "q18_probe_groupjoin": 20 * n_ol + 16 * n_o + 16 * n_o,
-        "q18_having_compact": 16 * n_o + 28 * n_o + 16 * n_pass + 4 * n_pass + 40 * n_pass,
+        "q18_init": slot_b * (slots_o + slots_c),               # empty the join indexes
+        # keys in, accumulators zeroed, one slot written per build row
+        "q18_build": 12 * n_o + 12 * n_c + 16 * n_o + slot_b * (n_o + n_c),
+        # order_line keys + amounts; per order one index slot and the accumulator read + write
+        "q18_probe_groupjoin": 20 * n_ol + slot_b * n_o + 16 * n_o + 16 * n_o,
+        # acc + orders columns in; per result row a customer slot + c_last lookup, 40 B out
+        "q18_having_compact": 16 * n_o + 28 * n_o + (slot_b + 4) * n_pass + 40 * n_pass,
         # ORDER BY v1 (H2TAP_ORDER=v1): (key, row id) sort, random row gather at emit
         "q18_sort_keys_hist": (32 + 8 + 8 + 4) * n_pass,   # rows + amounts -> keys + row ids
         # ORDER BY v2 (default): count matrix + scatter computing keys + chunked local sort
@@ -223,6 +241,8 @@ def main():
     n_ol = len(tables["order_line"]["ol_w_id"])
     n_o = len(tables["orders"]["o_id"])
     n_c = len(tables["customer"]["c_id"])
+    box = (key_box(tables["orders"], ("o_w_id", "o_d_id", "o_id")),
+           key_box(tables["customer"], ("c_w_id", "c_d_id", "c_id")))
     pinned = {t: {c: torch.from_numpy(v).pin_memory() for c, v in cols.items()} for t, cols in hot.items()}
     h2d_bytes = sum(v.numel() * v.element_size() for cols in pinned.values() for v in cols.values())
     epoch = 1
@@ -247,8 +267,12 @@ def main():
         for (name, _, _), r in zip(plans, rs):
             out[name] = (r.device_ms, r.kernels if flags & h.H2TAP_QUERY_PROFILE else [], r.nrows,
                          r.kernel_launches)
+            if name == "q18":
+                dense_seen.append(r.plan_flags == 3)  # both join indexes perfect-hash
             h.h2tap_free(r)
         return out
+
+    dense_seen = []
 
     dev_flags = h.H2TAP_RESULT_DEVICE
     prof_flags = h.H2TAP_RESULT_DEVICE | h.H2TAP_QUERY_PROFILE
@@ -301,6 +325,7 @@ def main():
     rows_total = 3 * n_ol * world  # weak scaling: every rank holds the same-sized shard
     value = rows_total / (step_ms / 1e3)
 
+    plan_dense = bool(dense_seen) and all(dense_seen)
     # ---- roofline for the dominant kernel (largest share of the step)
     kavg = {k: float(np.mean(v)) for k, v in kern.items()}
     sort_passes = ("v1" if os.environ.get("H2TAP_ORDER") == "v1"
@@ -309,7 +334,7 @@ def main():
     peak, peak_src = peaks()
     roof = None
     if dominant:
-        b = alg_bytes(dominant, n_ol, n_o, n_c, n_pass, sort_passes)
+        b = alg_bytes(dominant, n_ol, n_o, n_c, n_pass, sort_passes, box if plan_dense else None)
         if b:
             ach = b / (kavg[dominant] / 1e3) / 1e9
             tr = ncu_traffic().get(dominant)
@@ -320,7 +345,7 @@ def main():
                     "timing": "CUDA events on the engine stream, instrumented pass of the same K steps"}
     kernels_summary = {}
     for k, v in kavg.items():
-        b = alg_bytes(k, n_ol, n_o, n_c, n_pass, sort_passes)
+        b = alg_bytes(k, n_ol, n_o, n_c, n_pass, sort_passes, box if plan_dense else None)
         kernels_summary[k] = {"ms": round(v, 5), "share": round(v / step_ms_local, 4)}
         if b:
             kernels_summary[k]["GB/s"] = round(b / (v / 1e3) / 1e9, 1)
