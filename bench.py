@@ -322,7 +322,10 @@ def main():
     if world > 1:
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
     step_ms = float(t.item())
-    rows_total = 3 * n_ol * world  # weak scaling: every rank holds the same-sized shard
+    nt = torch.tensor([n_ol], dtype=torch.float64, device="cuda")
+    if world > 1:  # weak scaling: every rank holds its own shard of W warehouses
+        dist.all_reduce(nt, op=dist.ReduceOp.SUM)
+    rows_total = 3 * int(nt.item())  # order_line rows all ranks scanned, x3 queries
     value = rows_total / (step_ms / 1e3)
 
     plan_dense = bool(dense_seen) and all(dense_seen)
@@ -376,20 +379,24 @@ def main():
     # lent to the DMA and not modified), so step k's 1.2 GB upload (copy stream)
     # overlaps step k-1's result read-back (D2H, the other PCIe direction) and the queries; each
     # batch runs on the latest PUBLISHED epoch (k or k-1, reported per step) — double buffering
+    # (one rank only: with world > 1 the ranks could publish different epochs and a collective
+    # query must see one epoch everywhere)
     h.h2tap_sync(eng)
     barrier()
     lag = []
-    t0 = time.perf_counter()
-    for _ in range(e2e_steps):
-        epoch += 1
-        h.h2tap_load_snapshot(eng, pinned, epoch, flags=h.H2TAP_LOAD_ASYNC | h.H2TAP_LOAD_BORROW)
-        for r in h.h2tap_run_queries(eng, [(plan, p, 0) for _, plan, p in plans]):
-            _ = r.columns[next(iter(r.columns))][:1].sum() if r.nrows else 0  # host read
-            lag.append(epoch - r.epoch)
-            h.h2tap_free(r)
-    h.h2tap_sync(eng)  # the last upload is inside the timed region too
+    e2e_pipe_s = float("inf")
+    if world == 1:
+        t0 = time.perf_counter()
+        for _ in range(e2e_steps):
+            epoch += 1
+            h.h2tap_load_snapshot(eng, pinned, epoch, flags=h.H2TAP_LOAD_ASYNC | h.H2TAP_LOAD_BORROW)
+            for r in h.h2tap_run_queries(eng, [(plan, p, 0) for _, plan, p in plans]):
+                _ = r.columns[next(iter(r.columns))][:1].sum() if r.nrows else 0  # host read
+                lag.append(epoch - r.epoch)
+                h.h2tap_free(r)
+        h.h2tap_sync(eng)  # the last upload is inside the timed region too
+        e2e_pipe_s = (time.perf_counter() - t0) / e2e_steps
     barrier()
-    e2e_pipe_s = (time.perf_counter() - t0) / e2e_steps
     te = torch.tensor([e2e_serial_s, e2e_pipe_s], dtype=torch.float64, device="cuda")
     if world > 1:
         dist.all_reduce(te, op=dist.ReduceOp.MAX)
@@ -418,7 +425,7 @@ def main():
                        "l2": ("inputs > L2; between steps (outside events) 512 MB written then 256 MB read to flush L2"
                               if flush is not None else "inputs > L2 (no flush)")},
             "latency_ms": {q: round(float(np.median(v)), 4) for q, v in per_query.items()},
-            "rows_per_s": {q: n_ol * world / (float(np.median(v)) / 1e3) for q, v in per_query.items()},
+            "rows_per_s": {q: rows_total / 3 / (float(np.median(v)) / 1e3) for q, v in per_query.items()},
             "q18_result_rows": n_pass,
             "roofline": roof,
             "kernels": kernels_summary,
@@ -426,7 +433,8 @@ def main():
             "e2e": {"value": rows_total / e2e_s, "unit": UNIT, "h2d_bytes_per_step": int(h2d_bytes),
                     "d2h_bytes_per_step": int(d2h), "ms_per_step": e2e_s * 1e3, "steps": e2e_steps,
                     "mode": "pipelined" if e2e_pipe_s <= e2e_serial_s else "serial",
-                    "serial_ms_per_step": e2e_serial_s * 1e3, "pipelined_ms_per_step": e2e_pipe_s * 1e3,
+                    "serial_ms_per_step": e2e_serial_s * 1e3,
+                    "pipelined_ms_per_step": e2e_pipe_s * 1e3 if world == 1 else None,
                     "pipelined_epoch_lag": sorted(set(lag)),
                     "how": "every step: full snapshot upload of the step's inputs from pinned host "
                            "buffers (h2tap_load_snapshot) + Q6/Q1/Q18 batch (h2tap_run_queries) + "
