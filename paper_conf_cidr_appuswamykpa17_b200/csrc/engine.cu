@@ -99,18 +99,39 @@ inline size_t type_size(uint32_t t) { return t == H2TAP_I32 ? 4 : 8; }
 constexpr uint64_t kPadRows = 64;  // over-allocation so 128-bit loads of the last tile stay in bounds
 
 // ============================================================ memory ===
+// Streams a snapshot buffer's release is ordered after (DevBuf with a stream-ordered free).
+struct FreeOrder {
+    cudaStream_t compute = nullptr, copy = nullptr, reaper = nullptr;
+};
+
 struct DevBuf {  // one device allocation; freed when the last View referencing it dies
     void *ptr = nullptr;
     size_t bytes = 0;
     int device = 0;
+    const FreeOrder *order = nullptr;  // null: cudaMalloc / cudaFree (synchronising)
     ~DevBuf() {
-        if (ptr) {
-            int cur;
-            cudaGetDevice(&cur);
-            cudaSetDevice(device);
+        if (!ptr) return;
+        int cur;
+        cudaGetDevice(&cur);
+        cudaSetDevice(device);
+        if (order) {
+            // stream-ordered: released to the pool once everything already enqueued on the
+            // compute and copy streams is done, on a third stream — no device-wide sync (a
+            // cudaFree would stall every query and upload in flight) and no false dependency
+            cudaEvent_t a, b;
+            cudaEventCreateWithFlags(&a, cudaEventDisableTiming);
+            cudaEventCreateWithFlags(&b, cudaEventDisableTiming);
+            cudaEventRecord(a, order->compute);
+            cudaEventRecord(b, order->copy);
+            cudaStreamWaitEvent(order->reaper, a, 0);
+            cudaStreamWaitEvent(order->reaper, b, 0);
+            cudaFreeAsync(ptr, order->reaper);
+            cudaEventDestroy(a);
+            cudaEventDestroy(b);
+        } else {
             cudaFree(ptr);
-            cudaSetDevice(cur);
         }
+        cudaSetDevice(cur);
     }
 };
 using DevBufP = std::shared_ptr<DevBuf>;
@@ -120,6 +141,18 @@ DevBufP dev_alloc(size_t bytes, int device) {
     b->device = device;
     b->bytes = bytes;
     CK(cudaMalloc(&b->ptr, bytes ? bytes : 16));
+    return b;
+}
+
+// Snapshot column buffers: from the device's memory pool in copy-stream order (their first
+// writer), released stream-ordered (above). The pool keeps freed memory (release threshold =
+// max), so a full reload that cannot reuse the spare costs no cudaMalloc either.
+DevBufP dev_alloc_ordered(size_t bytes, int device, const FreeOrder *order) {
+    auto b = std::make_shared<DevBuf>();
+    b->device = device;
+    b->bytes = bytes;
+    CK(cudaMallocAsync(&b->ptr, bytes ? bytes : 16, order->copy));
+    b->order = order;
     return b;
 }
 
@@ -337,6 +370,8 @@ struct h2tap_engine {
     bool cow_full = false;
     ncclComm_t comm = nullptr;
     cudaStream_t compute = nullptr, copy = nullptr;
+    cudaStream_t reaper = nullptr;  // stream-ordered frees of snapshot buffers
+    FreeOrder free_order;
     cudaEvent_t q_begin = nullptr, q_end = nullptr;
 
     std::mutex load_mu, query_mu, view_mu, pend_mu;
@@ -637,7 +672,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
                 // view references it any more, else allocate
                 DevBufP target;
                 if (cs.alt && cs.alt.use_count() == 1 && cs.alt->bytes >= need * es) target = cs.alt;
-                else target = dev_alloc(need * es + need * es / 8, e->device);
+                else target = dev_alloc_ordered(need * es + need * es / 8, e->device, &e->free_order);
                 cs.alt = cs.cur;
                 cs.alt_valid = false;
                 cs.cur = target;
@@ -646,7 +681,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
                 // grow: new buffer, device-to-device copy of the visible prefix; the old buffer
                 // stays alive for views that still reference it
                 const uint64_t cap = std::max<uint64_t>(need, (cs.cap_rows * 3) / 2);
-                DevBufP nb = dev_alloc(cap * es, e->device);
+                DevBufP nb = dev_alloc_ordered(cap * es, e->device, &e->free_order);
                 if (cs.cur && t.first_row)
                     CK(cudaMemcpyAsync(nb->ptr, cs.cur->ptr, t.first_row * es, cudaMemcpyDeviceToDevice, e->copy));
                 cs.alt.reset();
@@ -709,8 +744,8 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         const uint64_t n_rows = v->n[u.table_id];
         const uint64_t words = (cs.cap_rows + kCowPageRows * 32 - 1) / (kCowPageRows * 32);
         if (!cs.bits || cs.bits->bytes < words * 4) {
-            cs.bits = dev_alloc(words * 4, e->device);
-            cs.bits_next = dev_alloc(words * 4, e->device);
+            cs.bits = dev_alloc_ordered(words * 4, e->device, &e->free_order);
+            cs.bits_next = dev_alloc_ordered(words * 4, e->device, &e->free_order);
             cs.alt_valid = false;  // no record of where alt differs
         }
         uint32_t *next_bits = static_cast<uint32_t *>(cs.bits_next->ptr);
@@ -719,7 +754,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
             launch_cow_catchup(cs.alt->ptr, cs.cur->ptr, (uint32_t)es, static_cast<const uint32_t *>(cs.bits->ptr),
                                next_bits, words, cs.alt_synced, n_rows, pages_dev, e->num_sms, e->copy);
         } else {
-            if (!reuse) cs.alt = dev_alloc(cs.cap_rows * es, e->device);
+            if (!reuse) cs.alt = dev_alloc_ordered(cs.cap_rows * es, e->device, &e->free_order);
             if (n_rows) CK(cudaMemcpyAsync(cs.alt->ptr, cs.cur->ptr, n_rows * es, cudaMemcpyDeviceToDevice, e->copy));
             CK(cudaMemsetAsync(next_bits, 0, words * 4, e->copy));
             pend.full_copies += 1;
@@ -1791,6 +1826,14 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
 
         CK(cudaStreamCreateWithFlags(&e->compute, cudaStreamNonBlocking));
         CK(cudaStreamCreateWithFlags(&e->copy, cudaStreamNonBlocking));
+        CK(cudaStreamCreateWithFlags(&e->reaper, cudaStreamNonBlocking));
+        e->free_order = FreeOrder{e->compute, e->copy, e->reaper};
+        {   // keep freed pool memory cached (no release to the OS at stream syncs)
+            cudaMemPool_t pool;
+            CK(cudaDeviceGetDefaultMemPool(&pool, e->device));
+            uint64_t thr = UINT64_MAX;
+            CK(cudaMemPoolSetAttribute(pool, cudaMemPoolAttrReleaseThreshold, &thr));
+        }
         CK(cudaEventCreate(&e->q_begin));
         CK(cudaEventCreate(&e->q_end));
         CK(cudaMallocHost(&e->small_host, 256));
@@ -1826,7 +1869,7 @@ h2tap_status h2tap_reserve(h2tap_engine *e, uint32_t table_id, uint64_t rows) {
             ColState &cs = ts.col[c];
             if (!cs.cur || cs.cap_rows >= need) continue;
             const size_t es = type_size(kTypes[table_id][c]);
-            DevBufP nb = dev_alloc(need * es, e->device);
+            DevBufP nb = dev_alloc_ordered(need * es, e->device, &e->free_order);
             if (ts.loaded)
                 CK(cudaMemcpyAsync(nb->ptr, cs.cur->ptr, ts.loaded * es, cudaMemcpyDeviceToDevice, e->copy));
             cs.alt.reset();
@@ -2059,8 +2102,10 @@ void h2tap_close(h2tap_engine *e) {
     for (auto &t : e->tables) for (auto &c : t.col) { c.cur.reset(); c.alt.reset(); c.bits.reset(); c.bits_next.reset(); }
     e->arena.bufs.clear();
     e->load_arena.bufs.clear();
+    cudaStreamSynchronize(e->reaper);
     cudaStreamDestroy(e->compute);
     cudaStreamDestroy(e->copy);
+    cudaStreamDestroy(e->reaper);
     delete e;
 }
 

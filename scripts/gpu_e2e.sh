@@ -1,5 +1,7 @@
-# async borrowed loads: parity test + bench (e2e serial vs pipelined)
+# stream-ordered snapshot buffers: full GPU suite + bench e2e (serial vs pipelined), twice
 mkdir -p gpurun_out
-timeout 600 python -m pytest tests/test_gpu_parity.py -q -x --timeout 300 -k "async_borrowed or snapshot or concurrent" 2>&1 | tail -3
-timeout 600 python bench.py --steps 10 --warmup 3 --no-cpu-baseline 2>&1 | tail -1 > gpurun_out/bench_e2e.json
-python -c "import json; d=json.load(open('gpurun_out/bench_e2e.json')); print(d['ms_per_step'], d['e2e'])"
+timeout 900 python -m pytest tests -m gpu -q --timeout 400 -x 2>&1 | tail -2
+for v in 1 2; do
+  timeout 600 python bench.py --steps 10 --warmup 3 --no-cpu-baseline 2>&1 | tail -1 > gpurun_out/bench_e2e.json
+  python -c "import json; d=json.load(open('gpurun_out/bench_e2e.json')); e=d['e2e']; print('run$v', d['ms_per_step'], e['serial_ms_per_step'], e['pipelined_ms_per_step'], e['pipelined_epoch_lag'])"
+done

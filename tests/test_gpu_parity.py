@@ -414,7 +414,7 @@ def test_async_borrowed_pinned_loads(h):
              oracle.q18(ts, Q18_HAVING)) for ts in sets]
     e = h.h2tap_open(0)
     try:
-        h.h2tap_load_snapshot(e, pinned[0], 1)
+        h.h2tap_load_snapshot(e, pinned[1], 1)  # epoch k holds set k % 2
         seen = set()
         for ep in range(2, 10):
             h.h2tap_load_snapshot(e, pinned[ep % 2], ep, flags=h.H2TAP_LOAD_ASYNC | h.H2TAP_LOAD_BORROW)
