@@ -148,6 +148,8 @@ DevBufP dev_alloc(size_t bytes, int device) {
 // writer), released stream-ordered (above). The pool keeps freed memory (release threshold =
 // max), so a full reload that cannot reuse the spare costs no cudaMalloc either.
 DevBufP dev_alloc_ordered(size_t bytes, int device, const FreeOrder *order) {
+    static const bool pool = [] { const char *v = std::getenv("H2TAP_POOL"); return !(v && v[0] == '0'); }();
+    if (!pool) return dev_alloc(bytes, device);  // A/B: cudaMalloc / synchronising cudaFree
     auto b = std::make_shared<DevBuf>();
     b->device = device;
     b->bytes = bytes;
@@ -1833,6 +1835,11 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
             CK(cudaDeviceGetDefaultMemPool(&pool, e->device));
             uint64_t thr = UINT64_MAX;
             CK(cudaMemPoolSetAttribute(pool, cudaMemPoolAttrReleaseThreshold, &thr));
+            // never let an allocation on the copy stream wait for a pending free (that free waits
+            // for queries on the compute stream: refreshes would serialise behind queries, C5
+            // measured 8 -> 101 ms per refresh); reuse only memory whose free has completed
+            int no = 0;
+            CK(cudaMemPoolSetAttribute(pool, cudaMemPoolReuseAllowInternalDependencies, &no));
         }
         CK(cudaEventCreate(&e->q_begin));
         CK(cudaEventCreate(&e->q_end));
