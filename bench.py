@@ -145,6 +145,8 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None):
     return {
         "q6_scan_filter_sum": 20 * n_ol,
         "q1_scan_filter_groupby": 24 * n_ol,
+        # shared scan of the batch's Q6 and Q1: Q1's 4 columns once, both queries
+        "q61_shared_scan": 24 * n_ol,
         "q18_init": slot_b * (slots_o + slots_c),               # empty the join indexes
         # keys in, accumulators zeroed, one slot written per build row
         "q18_build": 12 * n_o + 12 * n_c + 16 * n_o + slot_b * (n_o + n_c),

@@ -367,6 +367,7 @@ struct h2tap_engine {
     // H2TAP_ZC_TMA=0 selects the LDG kernels
     bool zc_tma = true;
     int having_unroll = 2;  // H2TAP_HAVING_UNROLL (2 or 4): orders rows per thread in the HAVING pass
+    bool shared_scan = true;  // H2TAP_SHARED_SCAN=0: separate Q6 and Q1 scans in a batch (A/B)
     // in-place updates copy only the dirty pages into the shadow (H2TAP_COW=full: always copy the
     // whole column — the A/B baseline of scripts/cow_bench.py)
     bool cow_full = false;
@@ -859,6 +860,9 @@ struct QueryCtx {
     Q18Scratch q18{};
     Q18Plan *plan_dev = nullptr;
     Q18Zone zone{};                         // ORDER BY field bounds from the zone maps
+    int64_t shared_cutoff = 0;              // the paired Q1's cutoff (shared_scan == 1)
+    int shared_scan = 0;                    // 1: this Q6 runs the batch's shared Q6+Q1 scan;
+                                            // 2: this Q1's scan was done by it
     const Q18Row *rows = nullptr;
     const long long *amt = nullptr;
     const unsigned int *perm = nullptr;
@@ -892,6 +896,8 @@ void give_blocks_to_result(QueryCtx &q) {
 }
 
 // ---- Q6 (a2 + a7)
+void q1_tables(h2tap_engine *e, Q1Scratch &s);
+
 void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     const int T = H2TAP_T_ORDER_LINE;
     need_cols(v, T, {H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}, "Q6");
@@ -905,6 +911,16 @@ void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
                          : static_cast<long long *>(dev_block(e, q, 16));
     s.host_out = e->world > 1 ? nullptr : static_cast<long long *>(q.small_dev);
     q.q6_out = s.out;
+    if (q.shared_scan == 1) {  // one pass for this Q6 and the batch's Q1 (its tables filled here)
+        Q1Scratch t{};
+        q1_tables(e, t);
+        e->prof.run("q61_shared_scan", [&] {
+            launch_q61_tma(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
+                           colp<int32_t>(v, T, H2TAP_OL_QUANTITY), colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T],
+                           q.shared_cutoff, t, q.p[0], q.p[1], q.p[2], q.p[3], s, e->num_sms, e->compute);
+            CK(cudaGetLastError());
+        });
+    } else
     e->prof.run("q6_scan_filter_sum", [&] {
         (e->scan_tma && (e->zc_tma || !v.any_host(T, {H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT})) ? launch_q6_tma : launch_q6)(
             colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D), colp<int32_t>(v, T, H2TAP_OL_QUANTITY),
@@ -942,10 +958,8 @@ void finish_q6(h2tap_engine *e, QueryCtx &q) {
 // ---- Q1 (a3 + a7 + a8)
 constexpr size_t kQ1MaxGroups = kQ1GlobalSlots + kQ1Dense;
 
-void launch_q1_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
-    const int T = H2TAP_T_ORDER_LINE;
-    need_cols(v, T, {H2TAP_OL_NUMBER, H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}, "Q1");
-    Q1Scratch &s = q.q1;
+// Q1's aggregation tables (named arena buffers; they self-clean in q1_compact after each use).
+void q1_tables(h2tap_engine *e, Q1Scratch &s) {
     const bool fresh = !e->arena.bufs.count("q1.gtag");
     s.dense = static_cast<unsigned long long *>(e->arena.get("q1.dense", 8 * kQ1Dense * 3));
     s.gtag = static_cast<unsigned long long *>(e->arena.get("q1.gtag", 8ull * kQ1GlobalSlots));
@@ -953,6 +967,19 @@ void launch_q1_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.flags = static_cast<unsigned int *>(e->arena.get("q1.flags", 64));
     s.groups = static_cast<Q1Group *>(e->arena.get("q1.groups", sizeof(Q1Group) * kQ1MaxGroups));
     s.ngroups = static_cast<unsigned long long *>(e->arena.get("q1.ngroups", 64));
+    if (fresh) launch_q1_reset(s, e->compute);
+}
+
+// The columns a Q6 / Q1 scan reads are all in HBM (or the zero-copy TMA path is enabled).
+bool scan_tma_ok(h2tap_engine *e, const View &v, std::initializer_list<int> cols) {
+    return e->scan_tma && (e->zc_tma || !v.any_host(H2TAP_T_ORDER_LINE, cols));
+}
+
+void launch_q1_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
+    const int T = H2TAP_T_ORDER_LINE;
+    need_cols(v, T, {H2TAP_OL_NUMBER, H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}, "Q1");
+    Q1Scratch &s = q.q1;
+    q1_tables(e, s);
     // outputs go straight into per-query device blocks (they become the result's columns)
     s.o_key = static_cast<int32_t *>(dev_block(e, q, 4 * kQ1MaxGroups));
     s.o_qty = static_cast<long long *>(dev_block(e, q, 8 * kQ1MaxGroups));
@@ -960,7 +987,7 @@ void launch_q1_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.o_avg_qty = static_cast<double *>(dev_block(e, q, 8 * kQ1MaxGroups));
     s.o_avg_amt = static_cast<double *>(dev_block(e, q, 8 * kQ1MaxGroups));
     s.o_cnt = static_cast<long long *>(dev_block(e, q, 8 * kQ1MaxGroups));
-    if (fresh) launch_q1_reset(s, e->compute);  // tables self-clean afterwards (q1_compact)
+    if (q.shared_scan != 2)
     e->prof.run("q1_scan_filter_groupby", [&] {
         (e->scan_tma && (e->zc_tma || !v.any_host(T, {H2TAP_OL_NUMBER, H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT})) ? launch_q1_tma : launch_q1)(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
                   colp<int32_t>(v, T, H2TAP_OL_QUANTITY), colp<int64_t>(v, T, H2TAP_OL_AMOUNT), v.n[T],
@@ -1683,6 +1710,23 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
         v = e->published;
     }
     if (!v) return fail(H2TAP_EPLAN, "no snapshot has been published yet");
+    {   // shared scan: one Q6 followed by one Q1 in the batch, both on the TMA
+        // path: the Q6 launch runs one pass over Q1's columns that serves both queries
+        int i6 = -1, i1 = -1, n6 = 0, n1 = 0;
+        for (uint32_t i = 0; i < n; ++i) {
+            if (ctx[i].plan == H2TAP_Q6) { i6 = (int)i; ++n6; }
+            if (ctx[i].plan == H2TAP_Q1) { i1 = (int)i; ++n1; }
+        }
+        const int OL = H2TAP_T_ORDER_LINE;
+        const bool cols = v->n[OL] && v->col[OL][H2TAP_OL_NUMBER] && v->col[OL][H2TAP_OL_DELIVERY_D] &&
+                          v->col[OL][H2TAP_OL_QUANTITY] && v->col[OL][H2TAP_OL_AMOUNT];
+        if (e->shared_scan && n6 == 1 && n1 == 1 && i6 < i1 && cols &&
+            scan_tma_ok(e, *v, {H2TAP_OL_NUMBER, H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT})) {
+            ctx[i6].shared_scan = 1;
+            ctx[i6].shared_cutoff = ctx[i1].p[0];
+            ctx[i1].shared_scan = 2;
+        }
+    }
     bool profile = false;
     for (auto &q : ctx) profile |= (q.flags & H2TAP_QUERY_PROFILE) != 0;
     e->prof.reset(profile, e->compute);
@@ -1823,6 +1867,7 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         if (const char *ob = std::getenv("H2TAP_ORDER")) e->order_v1 = std::strcmp(ob, "v1") == 0;
         if (const char *z = std::getenv("H2TAP_ZC_TMA")) e->zc_tma = std::atoi(z) != 0;
         if (const char *hu = std::getenv("H2TAP_HAVING_UNROLL")) e->having_unroll = std::atoi(hu) == 4 ? 4 : 2;
+        if (const char *ss = std::getenv("H2TAP_SHARED_SCAN")) e->shared_scan = std::atoi(ss) != 0;
         if (const char *impl = std::getenv("H2TAP_PROBE")) e->probe_tma = std::strcmp(impl, "tma") == 0;
         if (const char *impl = std::getenv("H2TAP_COW")) e->cow_full = std::strcmp(impl, "full") == 0;
 

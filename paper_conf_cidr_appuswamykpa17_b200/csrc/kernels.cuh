@@ -53,6 +53,12 @@ void launch_q1(const int32_t *number, const int64_t *deliv, const int32_t *qty,
 void launch_q1_tma(const int32_t *number, const int64_t *deliv, const int32_t *qty,
                    const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int num_sms,
                    cudaStream_t st);  // same result, TMA-bulk staged, one block per SM
+// Shared scan of a batch's Q6 and Q1: one TMA pass over Q1's four columns fills
+// Q1's tables (as launch_q1_tma) and writes Q6's {revenue, count} (as launch_q6_tma).
+void launch_q61_tma(const int32_t *number, const int64_t *deliv, const int32_t *qty,
+                    const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int64_t d_lo,
+                    int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s6, int num_sms,
+                    cudaStream_t st);
 void launch_q1_compact(const Q1Scratch &s, cudaStream_t st);        // tables -> groups[], ngroups
 void launch_q1_merge(const Q1Group *all, uint64_t n, const Q1Scratch &s, cudaStream_t st);
 void launch_q1_emit(const Q1Scratch &s, uint64_t max_groups, cudaStream_t st);  // rank by key + AVG;

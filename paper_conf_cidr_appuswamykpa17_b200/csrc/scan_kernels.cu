@@ -467,16 +467,29 @@ struct Q1Stages {
     uint64_t full[kQ1Stages], empty[kQ1Stages];
 };
 
-__global__ void __launch_bounds__(kTmaThreads, 1)
+// kQ6: shared scan of a batch's Q6 and Q1 — Q6 reads a subset of Q1's columns
+// (ol_delivery_d, ol_quantity, ol_amount), so the same staged chunk also feeds Q6's predicate and
+// sum; the block tail adds Q6's reduction (as q6_tma_kernel). One pass over 24 B/row instead of
+// 20 + 24.
+// Shared-scan block: warps 0-7 Q1 (as above), warp 8 the producer, warps 9-12 Q6 on the same
+// staged chunks (registers only) — Q6 added to the Q1 warps' rows lengthened their dependent
+// shared-memory update chains (145 vs 117 us); separate warps run it alongside.
+constexpr int kQ6SideWarps = 4;
+constexpr int kQ61Threads = (kTmaConsumerWarps + 1 + kQ6SideWarps) * 32;
+template <bool kQ6>
+__global__ void __launch_bounds__(kQ6 ? kQ61Threads : kTmaThreads, 1)
 q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deliv,
               const int *__restrict__ qty, const long long *__restrict__ amt, uint64_t n,
-              long long cutoff, Q1Scratch g) {
+              long long cutoff, Q1Scratch g, Q6Pred pred6, long long *__restrict__ part6,
+              unsigned int *__restrict__ counter6, long long *__restrict__ out6,
+              long long *__restrict__ host_out6) {
     pdl_wait();
     pdl_trigger();
     extern __shared__ __align__(128) unsigned char smem_raw[];
     Q1Stages &P = *reinterpret_cast<Q1Stages *>(smem_raw);
     Q1Smem &sm = *reinterpret_cast<Q1Smem *>(smem_raw + sizeof(Q1Stages));
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    long long sum6 = 0, cnt6 = 0;  // kQ6 only
     if (tid < kQ1Threads) {
 #pragma unroll
         for (int k = 0; k < kQ1Dense; ++k) { sm.cnt[k][tid] = 0; sm.qty[k][tid] = 0; sm.amt[k][tid] = 0; }
@@ -487,7 +500,7 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
     if (tid == 0) {
         for (int s = 0; s < kQ1Stages; ++s) {
             mbar_init(&P.full[s], 1);
-            mbar_init(&P.empty[s], kTmaConsumerWarps);
+            mbar_init(&P.empty[s], kTmaConsumerWarps + (kQ6 ? kQ6SideWarps : 0));
         }
         fence_mbar_init();
         if (blockIdx.x == 0) *g.ngroups = 0;  // consumed by q1_compact (stream-ordered)
@@ -512,7 +525,25 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
                 bulk_g2s(P.qty[s], qty + r0, b4, &P.full[s], pol);
             }
         }
-    } else {  // consumers: 256 threads, 4 rows each per chunk (warp-uniform trip count)
+    } else if (kQ6 && warp > kTmaConsumerWarps) {  // Q6 side warps: 128 threads, 8 rows each
+        const int t6 = tid - (kTmaConsumerWarps + 1) * 32;
+        int it = 0;
+        for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
+            const int s = it % kQ1Stages;
+            mbar_wait(&P.full[s], (unsigned)(it / kQ1Stages) & 1u);
+            const unsigned rows = (unsigned)(n - c * kQ1Chunk < (uint64_t)kQ1Chunk ? n - c * kQ1Chunk
+                                                                                 : (uint64_t)kQ1Chunk);
+#pragma unroll 8
+            for (unsigned r = t6; r < rows; r += kQ6SideWarps * 32) {
+                const long long d = P.deliv[s][r];
+                const bool p6 = pred6(d, P.qty[s][r]);
+                sum6 += p6 ? P.amt[s][r] : 0;
+                cnt6 += p6;
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&P.empty[s]);
+        }
+    } else {  // Q1 consumers: 256 threads, 4 rows each per chunk (warp-uniform trip count)
         int it = 0;
         for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
             const int s = it % kQ1Stages;
@@ -543,6 +574,40 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
     }
     __syncthreads();
     q1_block_merge(sm, g, tid);
+    if (kQ6) {  // Q6: block reduction -> per-block partial -> last block folds (q6_tma_kernel)
+        constexpr int kW = kQ61Threads / 32;
+        __shared__ long long s_sum[kW], s_cnt[kW];
+        __shared__ bool s_last;
+        sum6 = warp_sum(sum6);
+        cnt6 = warp_sum(cnt6);
+        if (lane == 0) { s_sum[warp] = sum6; s_cnt[warp] = cnt6; }
+        __syncthreads();
+        if (tid == 0) {
+            long long S0 = 0, C0 = 0;
+            for (int w = 0; w < kW; ++w) { S0 += s_sum[w]; C0 += s_cnt[w]; }
+            part6[2 * blockIdx.x] = S0;
+            part6[2 * blockIdx.x + 1] = C0;
+            __threadfence();
+            s_last = atomicAdd(counter6, 1u) == gridDim.x - 1;
+        }
+        __syncthreads();
+        if (s_last && warp == 0) {
+            __threadfence();
+            long long ts = 0, tc = 0;
+            for (unsigned b = lane; b < gridDim.x; b += 32) {
+                ts += __ldcg(part6 + 2 * b);
+                tc += __ldcg(part6 + 2 * b + 1);
+            }
+            ts = warp_sum(ts);
+            tc = warp_sum(tc);
+            if (lane == 0) {
+                out6[0] = ts;
+                out6[1] = tc;
+                if (host_out6) { host_out6[0] = ts; host_out6[1] = tc; }
+                *counter6 = 0;
+            }
+        }
+    }
 }
 
 // Collect the dense and global tables into groups[] and clear them for the next query.
@@ -687,13 +752,32 @@ void launch_q1_tma(const int32_t *number, const int64_t *deliv, const int32_t *q
     const size_t smem = sizeof(Q1Stages) + sizeof(Q1Smem);
     static bool init = false;
     if (!init) {
-        cudaFuncSetAttribute(q1_tma_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        cudaFuncSetAttribute(q1_tma_kernel<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         init = true;
     }
     const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
     const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
-    launch_pdl(q1_tma_kernel, grid, kTmaThreads, smem, st, number, reinterpret_cast<const long long *>(deliv), qty,
-                                                   reinterpret_cast<const long long *>(amt), n, cutoff, s);
+    launch_pdl(q1_tma_kernel<false>, grid, kTmaThreads, smem, st, number, reinterpret_cast<const long long *>(deliv), qty,
+               reinterpret_cast<const long long *>(amt), n, cutoff, s, Q6Pred{0, 0, 0, 0}, nullptr, nullptr,
+               nullptr, nullptr);
+    count_launches(1);
+}
+
+void launch_q61_tma(const int32_t *number, const int64_t *deliv, const int32_t *qty,
+                    const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int64_t d_lo,
+                    int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s6, int num_sms,
+                    cudaStream_t st) {
+    const size_t smem = sizeof(Q1Stages) + sizeof(Q1Smem);
+    static bool init = false;
+    if (!init) {
+        cudaFuncSetAttribute(q1_tma_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        init = true;
+    }
+    const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
+    const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
+    launch_pdl(q1_tma_kernel<true>, grid, kQ61Threads, smem, st, number, reinterpret_cast<const long long *>(deliv),
+               qty, reinterpret_cast<const long long *>(amt), n, cutoff, s, Q6Pred{d_lo, d_hi, q_lo, q_hi},
+               s6.block_part, s6.done_counter, s6.out, s6.host_out);
     count_launches(1);
 }
 
