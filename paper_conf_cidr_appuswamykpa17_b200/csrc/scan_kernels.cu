@@ -458,7 +458,7 @@ q1_kernel(const int4 *__restrict__ number, const longlong2 *__restrict__ deliv,
 // columns into a 4-stage ring (96 KB) next to the 88 KB of aggregation tables; warps 0-7
 // aggregate exactly as q1_kernel does (thread-private dense slots, warp-aggregated sparse path).
 constexpr int kQ1Chunk = 1024;
-constexpr int kQ1Stages = 4;
+constexpr int kQ1Stages = 5;
 struct Q1Stages {
     long long deliv[kQ1Stages][kQ1Chunk];
     long long amt[kQ1Stages][kQ1Chunk];
@@ -525,24 +525,47 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
                 bulk_g2s(P.qty[s], qty + r0, b4, &P.full[s], pol);
             }
         }
-    } else if (kQ6 && warp > kTmaConsumerWarps) {  // Q6 side warps: 128 threads, 8 rows each
+    } else if (kQ6 && warp > kTmaConsumerWarps) {  // Q6 side warps: 128 threads, 4 row pairs each
+        // the predicate as two unsigned range tests (same result as Q6Pred: a NULL date is
+        // INT64_MIN, below every lower bound > INT64_MIN; an empty range passes nothing)
+        const long long dlo = pred6.d_lo > kNullTs ? pred6.d_lo : kNullTs + 1;
+        const unsigned long long dspan = pred6.d_hi > dlo ? (unsigned long long)pred6.d_hi - (unsigned long long)dlo : 0ull;
+        const bool qempty = pred6.q_lo > pred6.q_hi;
+        const unsigned long long qspan = (unsigned long long)pred6.q_hi - (unsigned long long)pred6.q_lo;
+        auto pass = [&](long long d, int q) {
+            return ((unsigned long long)d - (unsigned long long)dlo < dspan) &
+                   ((unsigned long long)(long long)q - (unsigned long long)pred6.q_lo <= qspan) & !qempty;
+        };
         const int t6 = tid - (kTmaConsumerWarps + 1) * 32;
+        unsigned int c32 = 0;
         int it = 0;
         for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
             const int s = it % kQ1Stages;
             mbar_wait(&P.full[s], (unsigned)(it / kQ1Stages) & 1u);
             const unsigned rows = (unsigned)(n - c * kQ1Chunk < (uint64_t)kQ1Chunk ? n - c * kQ1Chunk
                                                                                  : (uint64_t)kQ1Chunk);
-#pragma unroll 8
-            for (unsigned r = t6; r < rows; r += kQ6SideWarps * 32) {
-                const long long d = P.deliv[s][r];
-                const bool p6 = pred6(d, P.qty[s][r]);
-                sum6 += p6 ? P.amt[s][r] : 0;
-                cnt6 += p6;
+            if (rows == (unsigned)kQ1Chunk) {  // full chunk: 128-bit / 64-bit shared loads of pairs
+#pragma unroll
+                for (int k = 0; k < kQ1Chunk / (2 * kQ6SideWarps * 32); ++k) {
+                    const unsigned pr = t6 + k * kQ6SideWarps * 32;
+                    const longlong2 d2 = reinterpret_cast<const longlong2 *>(P.deliv[s])[pr];
+                    const longlong2 a2 = reinterpret_cast<const longlong2 *>(P.amt[s])[pr];
+                    const int2 q2 = reinterpret_cast<const int2 *>(P.qty[s])[pr];
+                    const bool p0 = pass(d2.x, q2.x), p1 = pass(d2.y, q2.y);
+                    sum6 += (p0 ? a2.x : 0) + (p1 ? a2.y : 0);
+                    c32 += (unsigned)p0 + (unsigned)p1;
+                }
+            } else {
+                for (unsigned r = t6; r < rows; r += kQ6SideWarps * 32) {
+                    const bool p0 = pass(P.deliv[s][r], P.qty[s][r]);
+                    sum6 += p0 ? P.amt[s][r] : 0;
+                    c32 += p0;
+                }
             }
             __syncwarp();
             if (lane == 0) mbar_arrive(&P.empty[s]);
         }
+        cnt6 = c32;
     } else {  // Q1 consumers: 256 threads, 4 rows each per chunk (warp-uniform trip count)
         int it = 0;
         for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
@@ -550,14 +573,28 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
             mbar_wait(&P.full[s], (unsigned)(it / kQ1Stages) & 1u);
             const unsigned rows = (unsigned)(n - c * kQ1Chunk < (uint64_t)kQ1Chunk ? n - c * kQ1Chunk
                                                                                  : (uint64_t)kQ1Chunk);
+            // all four rows' loads first: the stage and the tables share one shared-memory
+            // buffer, so loads after a table store would wait for it (possible aliasing)
+            constexpr int kU = kQ1Chunk / kQ1Threads;
+            int keys[kU], qs[kU];
+            long long ds[kU], as[kU];
 #pragma unroll
-            for (int u = 0; u < kQ1Chunk / kQ1Threads; ++u) {
+            for (int u = 0; u < kU; ++u) {
                 const unsigned r = u * kQ1Threads + tid;
                 const bool valid = r < rows;
-                const int key = valid ? P.number[s][r] : 0;
-                const long long d = valid ? P.deliv[s][r] : kNullTs;
-                const int q = valid ? P.qty[s][r] : 0;
-                const long long a = valid ? P.amt[s][r] : 0;
+                keys[u] = valid ? P.number[s][r] : 0;
+                ds[u] = valid ? P.deliv[s][r] : kNullTs;
+                qs[u] = valid ? P.qty[s][r] : 0;
+                as[u] = valid ? P.amt[s][r] : 0;
+            }
+#pragma unroll
+            for (int u = 0; u < kU; ++u) {
+                const unsigned r = u * kQ1Threads + tid;
+                const bool valid = r < rows;
+                const int key = keys[u];
+                const long long d = ds[u];
+                const int q = qs[u];
+                const long long a = as[u];
                 // WHERE ol_delivery_d > cutoff (NULL -> UNKNOWN -> excluded), GROUP BY ol_number
                 const bool pass = valid & (d != kNullTs) & (d > cutoff);
                 const bool sparse = pass & ((unsigned)key >= (unsigned)kQ1Dense);

@@ -18,14 +18,20 @@ ap.add_argument("--warehouses", type=int, default=100)
 ap.add_argument("--reps", type=int, default=2)
 ap.add_argument("--plans", default="6,1,18")
 ap.add_argument("--flags", type=int, default=h.H2TAP_RESULT_DEVICE)
+ap.add_argument("--single", action="store_true", help="one h2tap_run_query per plan instead of one "
+                "batch per rep (the bench's step is a batch: shared Q6+Q1 scan)")
 a = ap.parse_args()
 
 t = chgen.generate(1, a.warehouses + 1, seed=1, mode="spread")
 e = h.h2tap_open(0)
 h.h2tap_load_snapshot(e, h.hot_path_tables(t), 1)
+plans = [int(x) for x in a.plans.split(",")]
 for _ in range(a.reps):
-    for p in [int(x) for x in a.plans.split(",")]:
-        r = h.h2tap_run_query(e, p, flags=a.flags)
-        h.h2tap_free(r)
+    if a.single:
+        for p in plans:
+            h.h2tap_free(h.h2tap_run_query(e, p, flags=a.flags))
+    else:
+        for r in h.h2tap_run_queries(e, [(p, None, a.flags) for p in plans]):
+            h.h2tap_free(r)
 h.h2tap_close(e)
 print("done")
