@@ -178,6 +178,40 @@ def test_q1_sparse_group_keys(L):
         assert_q1(L.q(1, [cut]), oracle.q1(t, cut))
 
 
+@pytest.mark.parametrize("shared", ["1", "0"])
+def test_shared_q6_q1_scan(h, monkeypatch, shared):
+    """A batch with one Q6 before one Q1 runs one shared scan: random Q6 windows
+    and quantity ranges (incl. empty and inverted ones, bounds at INT64_MIN), random Q1 cutoffs,
+    ragged sizes and NULL dates, vs the oracle; H2TAP_SHARED_SCAN=0 runs the two scans."""
+    monkeypatch.setenv("H2TAP_SHARED_SCAN", shared)
+    e = h.h2tap_open(0)
+    try:
+        L = Loader(h, e)
+        rng = np.random.default_rng(57)
+        for n_keep in (100_003, 2049, 1023, 1):
+            t = chgen.generate(1, 3, seed=57)
+            t["order_line"] = {k: v[:n_keep].copy() for k, v in t["order_line"].items()}
+            L.load(t)
+            cases = [(Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI, Q1_CUTOFF),
+                     (-(2**63), 2**63 - 1, -(2**63), 2**63 - 1, -(2**63)),  # everything non-NULL
+                     (chgen.TS_2025, chgen.TS_1995, 1, 10, chgen.TS_2025),   # inverted / empty
+                     (chgen.TS_1995, chgen.TS_2025, 7, 3, chgen.TS_1995)]   # empty quantity range
+            for _ in range(3):
+                d_lo = int(rng.integers(chgen.TS_1995, chgen.TS_2025))
+                cases.append((d_lo, int(rng.integers(d_lo, chgen.TS_2025 + 10**12)), int(rng.integers(0, 6)),
+                              int(rng.integers(4, 12)), int(rng.integers(chgen.TS_1995, chgen.TS_2025))))
+            for d_lo, d_hi, q_lo, q_hi, cut in cases:
+                rs = h.h2tap_run_queries(e, [(6, [d_lo, d_hi, q_lo, q_hi], 0), (1, [cut], 0)])
+                g6, g1 = rs[0].to_numpy(), rs[1].to_numpy()
+                g6["_nulls"] = dict(rs[0].nulls)
+                for r in rs:
+                    h.h2tap_free(r)
+                assert_q6(g6, oracle.q6(t, d_lo, d_hi, q_lo, q_hi))
+                assert_q1(g1, oracle.q1(t, cut))
+    finally:
+        h.h2tap_close(e)
+
+
 def test_q6_quantity_and_null_edges(L):
     t = chgen.generate(1, 2, seed=4)
     L.load(t)
@@ -554,9 +588,23 @@ def test_full_size_w100_bench_config(h, w100):
     try:
         h.h2tap_load_snapshot(e, h.hot_path_tables(w100), 1)
         L = Loader(h, e)
-        assert_q6(L.q(6), oracle.q6(w100, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))
-        assert_q1(L.q(1), oracle.q1(w100, Q1_CUTOFF))
+        want6 = oracle.q6(w100, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI)
+        want1 = oracle.q1(w100, Q1_CUTOFF)
         want = oracle.q18(w100, Q18_HAVING)
+        # the bench's step: one batch, device-resident results (shared Q6+Q1 scan, PDL chain)
+        rs = h.h2tap_run_queries(e, [(6, None, h.H2TAP_RESULT_DEVICE), (1, None, h.H2TAP_RESULT_DEVICE),
+                                     (18, None, h.H2TAP_RESULT_DEVICE)])
+        got = []
+        for r in rs:
+            x = r.to_numpy()
+            x["_nulls"] = {k: (v.copy() if hasattr(v, "copy") else v) for k, v in r.nulls.items()}
+            got.append(x)
+            h.h2tap_free(r)
+        assert_q6(got[0], want6)
+        assert_q1(got[1], want1)
+        assert_q18(got[2], want)
+        assert_q6(L.q(6), want6)
+        assert_q1(L.q(1), want1)
         assert_q18(L.q(18, flags=h.H2TAP_QUERY_PROFILE), want)
         assert_q18(L.q(18, flags=HASH), want)
     finally:
