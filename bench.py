@@ -430,6 +430,10 @@ def main():
                        "warehouses_per_gpu": a.warehouses, "order_line_rows_per_gpu": n_ol,
                        "orders_rows_per_gpu": n_o, "customer_rows_per_gpu": n_c,
                        "queries_per_step": 3, "parallelism": f"row-sharded by warehouse x{world}",
+                       "scan_sharing": ("Q6 and Q1 of the batch share one pass over order_line "
+                                        "(latency_ms q6 includes it, q1 is its finalize; DESIGN.md "
+                                        "§4.5); every query computes its full result"
+                                        if os.environ.get("H2TAP_SHARED_SCAN", "1") != "0" else "off"),
                        "l2": ("inputs > L2; between steps (outside events) 512 MB written then 256 MB read to flush L2"
                               if flush is not None else "inputs > L2 (no flush)")},
             "latency_ms": {q: round(float(np.median(v)), 4) for q, v in per_query.items()},
