@@ -600,8 +600,9 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
             fetch(wi + gridDim.x);
             continue;
         }
-        int sb = 0;
-        while (sb < 10 && (m >> (sb + sub_log2)) > 0) ++sb;
+        // sub-bucket bits: the smallest sb with (m >> (sb + sub_log2)) == 0, at most 10
+        int sb = 32 - __clz(m) - sub_log2;
+        sb = sb < 0 ? 0 : sb > 10 ? 10 : sb;
         if (sb > shift) sb = shift;
         const int ssh = shift - sb;
         const unsigned int ns = 1u << sb, smask = ns - 1u;
@@ -661,9 +662,11 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
             const unsigned int sbk = (unsigned int)(kk >> ssh) & smask;
             const unsigned int s0 = S.sub[sbk], s1 = S.sub[sbk + 1];
             unsigned int rank = s0;
-            for (unsigned int j = s0; j < s1; ++j) {
-                const unsigned long long kj = S.k2[j], vj = S.v2[j];
-                rank += (kj < kk) | ((kj == kk) & ((vj < vv) | ((vj == vv) & (j < i))));
+            if (s1 - s0 > 1) {  // (a sub-bucket of one row: its rank is its offset)
+                for (unsigned int j = s0; j < s1; ++j) {
+                    const unsigned long long kj = S.k2[j], vj = S.v2[j];
+                    rank += (kj < kk) | ((kj == kk) & ((vj < vv) | ((vj == vv) & (j < i))));
+                }
             }
             S.k1[rank] = kk;
             S.v1[rank] = vv;
@@ -672,7 +675,9 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         const unsigned int cur_lo = lo, cur_m = m;
         fetch(wi + gridDim.x);  // next bucket's records in flight during the stores below
         for (unsigned int i = threadIdx.x; i <= ns; i += kBkThreads) S.sub[i] = 0;
-        for (unsigned int i = threadIdx.x; i < cur_m; i += kBkThreads) {  // decode + coalesced stores
+        // decode + coalesced stores, two adjacent output rows per thread (8-byte stores of the
+        // int32 columns, 16-byte of the int64 ones); an odd first / last row goes alone
+        auto store1 = [&](unsigned int i) {
             const CarryRow c = carry_decode(S.k1[i], S.v1[i], sp);
             const uint64_t j = cur_lo + i;
             dst.c_last[j] = c.c_last;
@@ -683,7 +688,25 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
             dst.amount_sum[j] = c.amount;
             dst.o_w_id[j] = c.o_w_id;
             dst.o_d_id[j] = c.o_d_id;
+        };
+        const unsigned int head = cur_lo & 1u;  // output row cur_lo + i is even for i = head
+        const unsigned int npair = (cur_m - head) >> 1;
+        for (unsigned int p = threadIdx.x; p < npair; p += kBkThreads) {
+            const unsigned int i = head + 2 * p;
+            const CarryRow a = carry_decode(S.k1[i], S.v1[i], sp);
+            const CarryRow b = carry_decode(S.k1[i + 1], S.v1[i + 1], sp);
+            const uint64_t j = cur_lo + i;
+            *reinterpret_cast<int2 *>(dst.c_last + j) = make_int2(a.c_last, b.c_last);
+            *reinterpret_cast<int2 *>(dst.c_id + j) = make_int2(a.c_id, b.c_id);
+            *reinterpret_cast<int2 *>(dst.o_id + j) = make_int2(a.o_id, b.o_id);
+            *reinterpret_cast<longlong2 *>(dst.o_entry_d + j) = make_longlong2(a.o_entry_d, b.o_entry_d);
+            *reinterpret_cast<int2 *>(dst.o_ol_cnt + j) = make_int2(a.o_ol_cnt, b.o_ol_cnt);
+            *reinterpret_cast<longlong2 *>(dst.amount_sum + j) = make_longlong2(a.amount, b.amount);
+            *reinterpret_cast<int2 *>(dst.o_w_id + j) = make_int2(a.o_w_id, b.o_w_id);
+            *reinterpret_cast<int2 *>(dst.o_d_id + j) = make_int2(a.o_d_id, b.o_d_id);
         }
+        if (threadIdx.x == kBkThreads - 1 && head) store1(0);
+        if (threadIdx.x == kBkThreads - 2 && ((cur_m - head) & 1u)) store1(cur_m - 1);
         __syncthreads();
     }
 }
