@@ -543,13 +543,18 @@ template <int kLsCap> struct LsSmem {
 };
 
 // carry mode: 64-bit second words instead of 32-bit row ids (2 048 rows: 72 KB, 3 blocks/SM)
+// (records stay where they were loaded; the sort moves 16-bit indices: 48 KB for 2 048 rows,
+// 4 blocks per SM)
 template <int kCap> struct LcSmem {
-    unsigned long long k1[kCap], k2[kCap], v1[kCap], v2[kCap];
+    ulonglong2 rec[kCap];             // the bucket's records, load order
+    unsigned short idx[kCap];         // record ids grouped by sub-bucket
+    unsigned short srt[kCap];         // record ids in sorted order
     unsigned int sub[kLsSubMax + 1];
     unsigned int cur[kLsSubMax];
     unsigned int wsum[kBkThreads / 32];
 };
-constexpr int kLcCapLarge = 6144;  // carry records per bucket in the large instance (~197 KB)
+static_assert(kLsCapLarge <= 65536, "16-bit record ids");
+constexpr int kLcCapLarge = 8192;  // carry records per bucket in the large instance (~172 KB)
 
 // Per-bucket sort of carry records (same sub-bucket + rank scheme as the row-id body below,
 // 128-bit compares, no tie-fix) and the emit: every output column is decoded from the record,
@@ -610,15 +615,13 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         for (int u = 0; u < kPre; ++u) {
             const unsigned int i = threadIdx.x + u * kBkThreads;
             if (i < m) {
-                S.k1[i] = pre[u].x;
-                S.v1[i] = pre[u].y;
+                S.rec[i] = pre[u];
                 atomicAdd(&S.sub[(unsigned int)(pre[u].x >> ssh) & smask], 1u);
             }
         }
         for (unsigned int i = threadIdx.x + kPre * kBkThreads; i < m; i += kBkThreads) {  // rest
             const ulonglong2 r = __ldcs(kv + lo + i);
-            S.k1[i] = r.x;
-            S.v1[i] = r.y;
+            S.rec[i] = r;
             atomicAdd(&S.sub[(unsigned int)(r.x >> ssh) & smask], 1u);
         }
         __syncthreads();
@@ -651,25 +654,24 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         }
         __syncthreads();
         for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
-            const unsigned long long kk = S.k1[i];
+            const unsigned long long kk = S.rec[i].x;
             const unsigned int p = atomicAdd(&S.cur[(unsigned int)(kk >> ssh) & smask], 1u);
-            S.k2[p] = kk;
-            S.v2[p] = S.v1[i];
+            S.idx[p] = (unsigned short)i;
         }
         __syncthreads();
-        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {  // rank -> sorted smem
-            const unsigned long long kk = S.k2[i], vv = S.v2[i];
-            const unsigned int sbk = (unsigned int)(kk >> ssh) & smask;
+        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {  // rank -> sorted order
+            const unsigned int me = S.idx[i];
+            const ulonglong2 r = S.rec[me];
+            const unsigned int sbk = (unsigned int)(r.x >> ssh) & smask;
             const unsigned int s0 = S.sub[sbk], s1 = S.sub[sbk + 1];
             unsigned int rank = s0;
             if (s1 - s0 > 1) {  // (a sub-bucket of one row: its rank is its offset)
                 for (unsigned int j = s0; j < s1; ++j) {
-                    const unsigned long long kj = S.k2[j], vj = S.v2[j];
-                    rank += (kj < kk) | ((kj == kk) & ((vj < vv) | ((vj == vv) & (j < i))));
+                    const ulonglong2 o = S.rec[S.idx[j]];
+                    rank += (o.x < r.x) | ((o.x == r.x) & ((o.y < r.y) | ((o.y == r.y) & (j < i))));
                 }
             }
-            S.k1[rank] = kk;
-            S.v1[rank] = vv;
+            S.srt[rank] = (unsigned short)me;
         }
         __syncthreads();
         const unsigned int cur_lo = lo, cur_m = m;
@@ -678,7 +680,8 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         // decode + coalesced stores, two adjacent output rows per thread (8-byte stores of the
         // int32 columns, 16-byte of the int64 ones); an odd first / last row goes alone
         auto store1 = [&](unsigned int i) {
-            const CarryRow c = carry_decode(S.k1[i], S.v1[i], sp);
+            const ulonglong2 r = S.rec[S.srt[i]];
+            const CarryRow c = carry_decode(r.x, r.y, sp);
             const uint64_t j = cur_lo + i;
             dst.c_last[j] = c.c_last;
             dst.c_id[j] = c.c_id;
@@ -693,8 +696,9 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         const unsigned int npair = (cur_m - head) >> 1;
         for (unsigned int p = threadIdx.x; p < npair; p += kBkThreads) {
             const unsigned int i = head + 2 * p;
-            const CarryRow a = carry_decode(S.k1[i], S.v1[i], sp);
-            const CarryRow b = carry_decode(S.k1[i + 1], S.v1[i + 1], sp);
+            const ulonglong2 ra = S.rec[S.srt[i]], rb = S.rec[S.srt[i + 1]];
+            const CarryRow a = carry_decode(ra.x, ra.y, sp);
+            const CarryRow b = carry_decode(rb.x, rb.y, sp);
             const uint64_t j = cur_lo + i;
             *reinterpret_cast<int2 *>(dst.c_last + j) = make_int2(a.c_last, b.c_last);
             *reinterpret_cast<int2 *>(dst.c_id + j) = make_int2(a.c_id, b.c_id);
@@ -717,7 +721,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
 // capacity in big[1..]; the large instance walks only that queue.
 // kPairs: k holds interleaved 16-byte (key, row id) pairs (v2 scatter), v is unused.
 template <int kLsCap, int kMin, bool kPairs = false>
-__global__ void __launch_bounds__(kBkThreads, 3)
+__global__ void __launch_bounds__(kBkThreads, 4)
 bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigned int *__restrict__ v,
                          const unsigned int *__restrict__ offset, int nb,
                          const Q18Plan *__restrict__ plan, const Q18Row *__restrict__ rows,
@@ -731,7 +735,10 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
             reinterpret_cast<const ulonglong2 *>(k), offset, nb, plan, dst, flag, big, smem_raw, sub_log2);
         return;
     }
-    LsSmem<kLsCap> &S = *reinterpret_cast<LsSmem<kLsCap> *>(smem_raw);
+    // row-id path: the v2 small instance holds 1 536 rows (LsSmem<1536> fits the 48 KB of the
+    // carry layout, so both run 4 blocks per SM); larger buckets go to the large instance
+    constexpr int kRowCap = (kPairs && kMin == 0 && kLsCap == 2048) ? 1536 : kLsCap;
+    LsSmem<kRowCap> &S = *reinterpret_cast<LsSmem<kRowCap> *>(smem_raw);
     const int shift = plan->shift;
     const Q18SortSpec sp = plan->spec;
     const bool tiefix = plan->tiefix != 0;
@@ -743,7 +750,7 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
         const int b = kMin > 0 ? (int)big[1 + wi] : wi;
         const unsigned int lo = offset[b], m = offset[b + 1] - lo;
         if (m == 0) continue;
-        if (m > (unsigned)kLsCap) {
+        if (m > (unsigned)kRowCap) {
             if (threadIdx.x == 0) {
                 if (kMin > 0) atomicOr(flag, 2u);                 // too big even for shared memory
                 else big[1 + atomicAdd(big, 1u)] = (unsigned)b;   // hand over to the large instance
@@ -915,8 +922,8 @@ constexpr int kObThreads = 1024;   // hist / scatter: 2 blocks of 32 warps per S
 constexpr int kObCap = kLsCapSmall;  // per-bucket sort capacity: 2 048 rows (56 KB, 3 blocks/SM);
                                      // 4 096 (2 blocks/SM) with ~730-row buckets measured slower
 // dynamic shared memory of the v2 emit instances: row-id or carry layout, whichever is larger
-constexpr size_t kObSmem = sizeof(LsSmem<kObCap>) > sizeof(LcSmem<kObCap>) ? sizeof(LsSmem<kObCap>)
-                                                                           : sizeof(LcSmem<kObCap>);
+constexpr size_t kObSmem = sizeof(LsSmem<1536>) > sizeof(LcSmem<kObCap>) ? sizeof(LsSmem<1536>)
+                                                                         : sizeof(LcSmem<kObCap>);
 constexpr size_t kObSmemLarge = sizeof(LsSmem<kLsCapLarge>) > sizeof(LcSmem<kLcCapLarge>)
                                     ? sizeof(LsSmem<kLsCapLarge>) : sizeof(LcSmem<kLcCapLarge>);
 
@@ -1199,7 +1206,7 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
     end();
     // per-bucket shared-memory sort + tie-fix + emit: the v1 kernels on the (key, row id) pairs
     begin("q18_bucket_sort_emit");
-    const unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
+    const unsigned lb = (unsigned)nb < (unsigned)num_sms * 4 ? (unsigned)nb : (unsigned)num_sms * 4;
     launch_pdl(bucket_local_emit_kernel<kObCap, 0, true>, lb, kBkThreads, kObSmem, st,
         s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2);
     count_launches(1);
