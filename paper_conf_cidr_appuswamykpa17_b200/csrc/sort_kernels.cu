@@ -979,7 +979,7 @@ ob_hist_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ am
 // Column scans of the [G][nb] matrix: a block owns 32 buckets (lane); the [G][32] tile is staged
 // in shared memory with independent coalesced loads, scanned per column, written back. The last
 // block scans the bucket totals into bucket offsets.
-constexpr int kScanWarps = 8;
+constexpr int kScanWarps = 32;
 __global__ void __launch_bounds__(32 * kScanWarps)
 ob_scan_kernel(unsigned int *__restrict__ mat, int G, int nb, unsigned int *__restrict__ count,
                unsigned int *__restrict__ offset, unsigned int *ticket) {
