@@ -152,19 +152,22 @@ __device__ __forceinline__ void probe_lane_group(const Q18Scratch &s, const Key3
         const bool f[4] = {b1, b2, b3, !next_cont};
         const long long fs[4] = {s0 + carry_s, s1 + (b1 ? 0 : carry_s), s2 + ((b1 | b2) ? 0 : carry_s), is};
         const unsigned fc[4] = {c0 + carry_c, c1 + (b1 ? 0 : carry_c), c2 + ((b1 | b2) ? 0 : carry_c), ic};
-        unsigned int row[4];
-#pragma unroll
-        for (int j = 0; j < 4; ++j) row[j] = f[j] ? jx_lookup(s.jo, k[j].w, k[j].d, k[j].o) : kNoRow;
-        if (kFilter) {
-#pragma unroll
-            for (int j = 0; j < 4; ++j) row[j] = keep_row<true>(s, row[j]);
-        }
-#pragma unroll
-        for (int j = 0; j < 4; ++j)
-            if (row[j] != kNoRow) {
-                atomicAdd(reinterpret_cast<unsigned long long *>(&s.acc[row[j]].sum), (unsigned long long)fs[j]);
-                atomicAdd(&s.acc[row[j]].cnt, fc[j]);
+        // one probe + two atomics per run end, looping over this lane's run ends only (a lane
+        // holds at most one end inside plus the flush of its last run: the warp iterates 1-2
+        // times instead of executing four predicated probes)
+        unsigned em = (unsigned)f[0] | ((unsigned)f[1] << 1) | ((unsigned)f[2] << 2) | ((unsigned)f[3] << 3);
+        while (em) {
+            const int j = __ffs(em) - 1;
+            em &= em - 1;
+            const Key3 kj = j == 0 ? k[0] : j == 1 ? k[1] : j == 2 ? k[2] : k[3];
+            const long long sj = j == 0 ? fs[0] : j == 1 ? fs[1] : j == 2 ? fs[2] : fs[3];
+            const unsigned cj = j == 0 ? fc[0] : j == 1 ? fc[1] : j == 2 ? fc[2] : fc[3];
+            const unsigned int row = keep_row<kFilter>(s, jx_lookup(s.jo, kj.w, kj.d, kj.o));
+            if (row != kNoRow) {
+                atomicAdd(reinterpret_cast<unsigned long long *>(&s.acc[row].sum), (unsigned long long)sj);
+                atomicAdd(&s.acc[row].cnt, cj);
             }
+        }
 }
 
 template <bool kFilter>
