@@ -260,13 +260,14 @@ constexpr int kQ1Threads = 256;
 constexpr int kQ1Unroll = 2;   // 4-row vectors per lane per warp iteration
 constexpr int kQ1Sparse = 256; // per-block shared hash slots for keys outside [0, kQ1Dense)
 
-struct Q1Smem {
-    unsigned int cnt[kQ1Dense][kQ1Threads];  // [key][thread]: lane-distinct banks, no conflicts
-    long long qty[kQ1Dense][kQ1Threads];
-    long long amt[kQ1Dense][kQ1Threads];
+template <int kT> struct Q1SmemT {       // kT aggregating threads
+    unsigned int cnt[kQ1Dense][kT];          // [key][thread]: lane-distinct banks, no conflicts
+    long long qty[kQ1Dense][kT];
+    long long amt[kQ1Dense][kT];
     unsigned long long stag[kQ1Sparse];      // 0 = empty, else (1<<32 | (u32)key)
     unsigned long long sacc[kQ1Sparse][3];
 };
+using Q1Smem = Q1SmemT<kQ1Threads>;
 
 __device__ __forceinline__ unsigned int hash32(unsigned int x) {
     x ^= x >> 16; x *= 0x7feb352dU; x ^= x >> 15; x *= 0x846ca68bU; x ^= x >> 16;
@@ -289,7 +290,8 @@ __device__ void q1_global_add(const Q1Scratch &g, unsigned long long tag, unsign
     atomicOr(g.flags, 1u);  // more distinct groups than kQ1GlobalSlots: reported as ENOMEM
 }
 
-__device__ void q1_sparse_add(Q1Smem &sm, const Q1Scratch &g, int key, unsigned long long c,
+template <class Sm>
+__device__ void q1_sparse_add(Sm &sm, const Q1Scratch &g, int key, unsigned long long c,
                               long long q, long long a) {
     const unsigned long long tag = (1ull << 32) | (unsigned int)key;
     unsigned int h = hash32((unsigned int)key) & (kQ1Sparse - 1);
@@ -309,7 +311,8 @@ __device__ void q1_sparse_add(Q1Smem &sm, const Q1Scratch &g, int key, unsigned 
 // Warp-aggregated shared-memory atomics: lanes with the same key are grouped (one ballot per
 // distinct key present in the warp), their values are reduced with shuffles, and only the
 // group leader touches the hash table. Called convergently by all 32 lanes.
-__device__ __forceinline__ void q1_sparse_warp(Q1Smem &sm, const Q1Scratch &g, bool need, int key,
+template <class Sm>
+__device__ __forceinline__ void q1_sparse_warp(Sm &sm, const Q1Scratch &g, bool need, int key,
                                                long long q, long long a) {
     const int lane = threadIdx.x & 31;
     unsigned int pend = __ballot_sync(kFull, need);
@@ -328,12 +331,13 @@ __device__ __forceinline__ void q1_sparse_warp(Q1Smem &sm, const Q1Scratch &g, b
 
 // Block end: dense keys, one warp per key, one global atomic per (key, accumulator) per block;
 // the block's sparse table into the global table. Threads tid < kQ1Threads take part.
-__device__ void q1_block_merge(Q1Smem &sm, const Q1Scratch &g, int tid) {
-    if (tid >= kQ1Threads) return;
+template <int kT = kQ1Threads>
+__device__ void q1_block_merge(Q1SmemT<kT> &sm, const Q1Scratch &g, int tid) {
+    if (tid >= kT) return;
     const int lane = tid & 31, warp = tid >> 5;
-    for (int k = warp; k < kQ1Dense; k += kQ1Threads / 32) {
+    for (int k = warp; k < kQ1Dense; k += kT / 32) {
         long long c = 0, q = 0, a = 0;
-        for (int t = lane; t < kQ1Threads; t += 32) { c += sm.cnt[k][t]; q += sm.qty[k][t]; a += sm.amt[k][t]; }
+        for (int t = lane; t < kT; t += 32) { c += sm.cnt[k][t]; q += sm.qty[k][t]; a += sm.amt[k][t]; }
         c = warp_sum(c); q = warp_sum(q); a = warp_sum(a);
         if (lane == 0 && c) {
             atomicAdd(g.dense + 3 * k + 0, (unsigned long long)c);
@@ -341,7 +345,7 @@ __device__ void q1_block_merge(Q1Smem &sm, const Q1Scratch &g, int tid) {
             atomicAdd(g.dense + 3 * k + 2, (unsigned long long)a);
         }
     }
-    for (int s = tid; s < kQ1Sparse; s += kQ1Threads)
+    for (int s = tid; s < kQ1Sparse; s += kT)
         if (sm.stag[s]) q1_global_add(g, sm.stag[s], sm.sacc[s][0], (long long)sm.sacc[s][1],
                                       (long long)sm.sacc[s][2]);
 }
@@ -458,13 +462,19 @@ q1_kernel(const int4 *__restrict__ number, const longlong2 *__restrict__ deliv,
 // columns into a 4-stage ring (96 KB) next to the 88 KB of aggregation tables; warps 0-7
 // aggregate exactly as q1_kernel does (thread-private dense slots, warp-aggregated sparse path).
 constexpr int kQ1Chunk = 1024;
-constexpr int kQ1Stages = 5;
-struct Q1Stages {
-    long long deliv[kQ1Stages][kQ1Chunk];
-    long long amt[kQ1Stages][kQ1Chunk];
-    int number[kQ1Stages][kQ1Chunk];
-    int qty[kQ1Stages][kQ1Chunk];
-    uint64_t full[kQ1Stages], empty[kQ1Stages];
+template <int kS> struct Q1StagesT {
+    long long deliv[kS][kQ1Chunk];
+    long long amt[kS][kQ1Chunk];
+    int number[kS][kQ1Chunk];
+    int qty[kS][kQ1Chunk];
+    uint64_t full[kS], empty[kS];
+};
+// Q1 alone: 8 aggregating warps, 5 stages (208 KB). Shared with Q6: 12 aggregating warps (their
+// latency-bound slot updates were the shared pass's limit) and 4 stages (224 KB).
+template <bool kQ6> struct Q1TmaCfg {
+    static constexpr int kW = kQ6 ? 12 : kTmaConsumerWarps;  // aggregating warps
+    static constexpr int kT = kW * 32;
+    static constexpr int kS = kQ6 ? 4 : 5;                    // ring stages
 };
 
 // kQ6: shared scan of a batch's Q6 and Q1 — Q6 reads a subset of Q1's columns
@@ -475,7 +485,7 @@ struct Q1Stages {
 // staged chunks (registers only) — Q6 added to the Q1 warps' rows lengthened their dependent
 // shared-memory update chains (145 vs 117 us); separate warps run it alongside.
 constexpr int kQ6SideWarps = 4;
-constexpr int kQ61Threads = (kTmaConsumerWarps + 1 + kQ6SideWarps) * 32;
+constexpr int kQ61Threads = (Q1TmaCfg<true>::kW + 1 + kQ6SideWarps) * 32;
 template <bool kQ6>
 __global__ void __launch_bounds__(kQ6 ? kQ61Threads : kTmaThreads, 1)
 q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deliv,
@@ -486,28 +496,30 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
     pdl_wait();
     pdl_trigger();
     extern __shared__ __align__(128) unsigned char smem_raw[];
-    Q1Stages &P = *reinterpret_cast<Q1Stages *>(smem_raw);
-    Q1Smem &sm = *reinterpret_cast<Q1Smem *>(smem_raw + sizeof(Q1Stages));
+    using Cfg = Q1TmaCfg<kQ6>;
+    constexpr int kQ1W = Cfg::kW, kQ1T = Cfg::kT, kQ1Stages = Cfg::kS;
+    Q1StagesT<kQ1Stages> &P = *reinterpret_cast<Q1StagesT<kQ1Stages> *>(smem_raw);
+    Q1SmemT<kQ1T> &sm = *reinterpret_cast<Q1SmemT<kQ1T> *>(smem_raw + sizeof(Q1StagesT<kQ1Stages>));
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     long long sum6 = 0, cnt6 = 0;  // kQ6 only
-    if (tid < kQ1Threads) {
+    if (tid < kQ1T) {
 #pragma unroll
         for (int k = 0; k < kQ1Dense; ++k) { sm.cnt[k][tid] = 0; sm.qty[k][tid] = 0; sm.amt[k][tid] = 0; }
-        for (int s = tid; s < kQ1Sparse; s += kQ1Threads) {
+        for (int s = tid; s < kQ1Sparse; s += kQ1T) {
             sm.stag[s] = 0; sm.sacc[s][0] = 0; sm.sacc[s][1] = 0; sm.sacc[s][2] = 0;
         }
     }
     if (tid == 0) {
         for (int s = 0; s < kQ1Stages; ++s) {
             mbar_init(&P.full[s], 1);
-            mbar_init(&P.empty[s], kTmaConsumerWarps + (kQ6 ? kQ6SideWarps : 0));
+            mbar_init(&P.empty[s], kQ1W + (kQ6 ? kQ6SideWarps : 0));
         }
         fence_mbar_init();
         if (blockIdx.x == 0) *g.ngroups = 0;  // consumed by q1_compact (stream-ordered)
     }
     __syncthreads();
     const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
-    if (warp == kTmaConsumerWarps) {  // producer
+    if (warp == kQ1W) {  // producer
         if (lane == 0) {
             const uint64_t pol = policy_evict_first();
             int it = 0;
@@ -525,7 +537,7 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
                 bulk_g2s(P.qty[s], qty + r0, b4, &P.full[s], pol);
             }
         }
-    } else if (kQ6 && warp > kTmaConsumerWarps) {  // Q6 side warps: 128 threads, 4 row pairs each
+    } else if (kQ6 && warp > kQ1W) {  // Q6 side warps: 128 threads, 4 row pairs each
         // the predicate as two unsigned range tests (same result as Q6Pred: a NULL date is
         // INT64_MIN, below every lower bound > INT64_MIN; an empty range passes nothing)
         const long long dlo = pred6.d_lo > kNullTs ? pred6.d_lo : kNullTs + 1;
@@ -536,7 +548,7 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
             return ((unsigned long long)d - (unsigned long long)dlo < dspan) &
                    ((unsigned long long)(long long)q - (unsigned long long)pred6.q_lo <= qspan) & !qempty;
         };
-        const int t6 = tid - (kTmaConsumerWarps + 1) * 32;
+        const int t6 = tid - (kQ1W + 1) * 32;
         unsigned int c32 = 0;
         int it = 0;
         for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
@@ -575,12 +587,12 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
                                                                                  : (uint64_t)kQ1Chunk);
             // all four rows' loads first: the stage and the tables share one shared-memory
             // buffer, so loads after a table store would wait for it (possible aliasing)
-            constexpr int kU = kQ1Chunk / kQ1Threads;
+            constexpr int kU = (kQ1Chunk + kQ1T - 1) / kQ1T;
             int keys[kU], qs[kU];
             long long ds[kU], as[kU];
 #pragma unroll
             for (int u = 0; u < kU; ++u) {
-                const unsigned r = u * kQ1Threads + tid;
+                const unsigned r = u * kQ1T + tid;
                 const bool valid = r < rows;
                 keys[u] = valid ? P.number[s][r] : 0;
                 ds[u] = valid ? P.deliv[s][r] : kNullTs;
@@ -589,7 +601,7 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
             }
 #pragma unroll
             for (int u = 0; u < kU; ++u) {
-                const unsigned r = u * kQ1Threads + tid;
+                const unsigned r = u * kQ1T + tid;
                 const bool valid = r < rows;
                 const int key = keys[u];
                 const long long d = ds[u];
@@ -610,7 +622,7 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
         }
     }
     __syncthreads();
-    q1_block_merge(sm, g, tid);
+    q1_block_merge<kQ1T>(sm, g, tid);
     if (kQ6) {  // Q6: block reduction -> per-block partial -> last block folds (q6_tma_kernel)
         constexpr int kW = kQ61Threads / 32;
         __shared__ long long s_sum[kW], s_cnt[kW];
@@ -786,7 +798,8 @@ void launch_q1(const int32_t *number, const int64_t *deliv, const int32_t *qty,
 void launch_q1_tma(const int32_t *number, const int64_t *deliv, const int32_t *qty,
                    const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int num_sms,
                    cudaStream_t st) {
-    const size_t smem = sizeof(Q1Stages) + sizeof(Q1Smem);
+    using Cfg = Q1TmaCfg<false>;
+    const size_t smem = sizeof(Q1StagesT<Cfg::kS>) + sizeof(Q1SmemT<Cfg::kT>);
     static bool init = false;
     if (!init) {
         cudaFuncSetAttribute(q1_tma_kernel<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -804,7 +817,8 @@ void launch_q61_tma(const int32_t *number, const int64_t *deliv, const int32_t *
                     const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int64_t d_lo,
                     int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s6, int num_sms,
                     cudaStream_t st) {
-    const size_t smem = sizeof(Q1Stages) + sizeof(Q1Smem);
+    using Cfg = Q1TmaCfg<true>;
+    const size_t smem = sizeof(Q1StagesT<Cfg::kS>) + sizeof(Q1SmemT<Cfg::kT>);
     static bool init = false;
     if (!init) {
         cudaFuncSetAttribute(q1_tma_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
