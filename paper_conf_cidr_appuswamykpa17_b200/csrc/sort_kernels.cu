@@ -421,7 +421,8 @@ constexpr int kBkThreads = 256;
 constexpr int kBkItems = 16;                       // rows per thread in the scatter
 constexpr int kLsCapSmall = 2048;                  // rows per bucket: fast kernel (3 blocks/SM)
 constexpr int kLsCapLarge = 8192;                  // rows per bucket: large-bucket kernel
-constexpr int kLsSubMax = 1024;                    // max sub-buckets per bucket
+constexpr int kLsSubMax = 512;                     // max sub-buckets per bucket (4 per emit thread)
+constexpr int kEmThreads = 128;                    // per-bucket sort / emit block (8 blocks/SM)
 
 // 1. keys + histogram (+ bucket scan by the last block)
 __global__ void __launch_bounds__(kBkThreads)
@@ -539,7 +540,7 @@ template <int kLsCap> struct LsSmem {
     unsigned int v1[kLsCap], v2[kLsCap];
     unsigned int sub[kLsSubMax + 1];   // sub-bucket counts -> offsets
     unsigned int cur[kLsSubMax];       // sub-bucket cursors
-    unsigned int wsum[kBkThreads / 32];
+    unsigned int wsum[kEmThreads / 32];
 };
 
 // carry mode: 64-bit second words instead of 32-bit row ids (2 048 rows: 72 KB, 3 blocks/SM)
@@ -551,7 +552,7 @@ template <int kCap> struct LcSmem {
     unsigned short srt[kCap];         // record ids in sorted order
     unsigned int sub[kLsSubMax + 1];
     unsigned int cur[kLsSubMax];
-    unsigned int wsum[kBkThreads / 32];
+    unsigned int wsum[kEmThreads / 32];
 };
 static_assert(kLsCapLarge <= 65536, "16-bit record ids");
 constexpr int kLcCapLarge = 8192;  // carry records per bucket in the large instance (~172 KB)
@@ -561,7 +562,7 @@ constexpr int kLcCapLarge = 8192;  // carry records per bucket in the large inst
 // so the only global traffic is the bucket's records in and the result columns out. The next
 // bucket's first kPre * 256 records are loaded into registers while the current one is
 // decoded and stored, and its sub-bucket counters are cleared then too (one barrier less).
-constexpr int kPre = 2;
+constexpr int kPre = 3;
 template <int kCap, int kMin>
 __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ kv,
                                                 const unsigned int *__restrict__ offset, int nb,
@@ -593,11 +594,11 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         }
 #pragma unroll
         for (int u = 0; u < kPre; ++u) {
-            const unsigned int i = threadIdx.x + u * kBkThreads;
+            const unsigned int i = threadIdx.x + u * kEmThreads;
             if (i < m) pre[u] = __ldcs(kv + lo + i);
         }
     };
-    for (unsigned int i = threadIdx.x; i <= kLsSubMax; i += kBkThreads) S.sub[i] = 0;
+    for (unsigned int i = threadIdx.x; i <= kLsSubMax; i += kEmThreads) S.sub[i] = 0;
     fetch(blockIdx.x);
     __syncthreads();
     for (int wi = blockIdx.x; wi < nwork; wi += gridDim.x) {
@@ -607,19 +608,19 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         }
         // sub-bucket bits: the smallest sb with (m >> (sb + sub_log2)) == 0, at most 10
         int sb = 32 - __clz(m) - sub_log2;
-        sb = sb < 0 ? 0 : sb > 10 ? 10 : sb;
+        sb = sb < 0 ? 0 : sb > 9 ? 9 : sb;  // ns <= kLsSubMax
         if (sb > shift) sb = shift;
         const int ssh = shift - sb;
         const unsigned int ns = 1u << sb, smask = ns - 1u;
 #pragma unroll
         for (int u = 0; u < kPre; ++u) {
-            const unsigned int i = threadIdx.x + u * kBkThreads;
+            const unsigned int i = threadIdx.x + u * kEmThreads;
             if (i < m) {
                 S.rec[i] = pre[u];
                 atomicAdd(&S.sub[(unsigned int)(pre[u].x >> ssh) & smask], 1u);
             }
         }
-        for (unsigned int i = threadIdx.x + kPre * kBkThreads; i < m; i += kBkThreads) {  // rest
+        for (unsigned int i = threadIdx.x + kPre * kEmThreads; i < m; i += kEmThreads) {  // rest
             const ulonglong2 r = __ldcs(kv + lo + i);
             S.rec[i] = r;
             atomicAdd(&S.sub[(unsigned int)(r.x >> ssh) & smask], 1u);
@@ -650,16 +651,16 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
                 if (i < ns) { S.sub[i] = run; S.cur[i] = run; }
                 run += c[q];
             }
-            if (threadIdx.x == kBkThreads - 1) S.sub[ns] = run;
+            if (threadIdx.x == kEmThreads - 1) S.sub[ns] = run;
         }
         __syncthreads();
-        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
+        for (unsigned int i = threadIdx.x; i < m; i += kEmThreads) {
             const unsigned long long kk = S.rec[i].x;
             const unsigned int p = atomicAdd(&S.cur[(unsigned int)(kk >> ssh) & smask], 1u);
             S.idx[p] = (unsigned short)i;
         }
         __syncthreads();
-        for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {  // rank -> sorted order
+        for (unsigned int i = threadIdx.x; i < m; i += kEmThreads) {  // rank -> sorted order
             const unsigned int me = S.idx[i];
             const ulonglong2 r = S.rec[me];
             const unsigned int sbk = (unsigned int)(r.x >> ssh) & smask;
@@ -676,7 +677,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         __syncthreads();
         const unsigned int cur_lo = lo, cur_m = m;
         fetch(wi + gridDim.x);  // next bucket's records in flight during the stores below
-        for (unsigned int i = threadIdx.x; i <= ns; i += kBkThreads) S.sub[i] = 0;
+        for (unsigned int i = threadIdx.x; i <= ns; i += kEmThreads) S.sub[i] = 0;
         // decode + coalesced stores, two adjacent output rows per thread (8-byte stores of the
         // int32 columns, 16-byte of the int64 ones); an odd first / last row goes alone
         auto store1 = [&](unsigned int i) {
@@ -694,7 +695,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         };
         const unsigned int head = cur_lo & 1u;  // output row cur_lo + i is even for i = head
         const unsigned int npair = (cur_m - head) >> 1;
-        for (unsigned int p = threadIdx.x; p < npair; p += kBkThreads) {
+        for (unsigned int p = threadIdx.x; p < npair; p += kEmThreads) {
             const unsigned int i = head + 2 * p;
             const ulonglong2 ra = S.rec[S.srt[i]], rb = S.rec[S.srt[i + 1]];
             const CarryRow a = carry_decode(ra.x, ra.y, sp);
@@ -709,8 +710,8 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
             *reinterpret_cast<int2 *>(dst.o_w_id + j) = make_int2(a.o_w_id, b.o_w_id);
             *reinterpret_cast<int2 *>(dst.o_d_id + j) = make_int2(a.o_d_id, b.o_d_id);
         }
-        if (threadIdx.x == kBkThreads - 1 && head) store1(0);
-        if (threadIdx.x == kBkThreads - 2 && ((cur_m - head) & 1u)) store1(cur_m - 1);
+        if (threadIdx.x == kEmThreads - 1 && head) store1(0);
+        if (threadIdx.x == kEmThreads - 2 && ((cur_m - head) & 1u)) store1(cur_m - 1);
         __syncthreads();
     }
 }
@@ -721,7 +722,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
 // capacity in big[1..]; the large instance walks only that queue.
 // kPairs: k holds interleaved 16-byte (key, row id) pairs (v2 scatter), v is unused.
 template <int kLsCap, int kMin, bool kPairs = false>
-__global__ void __launch_bounds__(kBkThreads, 4)
+__global__ void __launch_bounds__(kEmThreads, 6)
 bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigned int *__restrict__ v,
                          const unsigned int *__restrict__ offset, int nb,
                          const Q18Plan *__restrict__ plan, const Q18Row *__restrict__ rows,
@@ -737,7 +738,7 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
     }
     // row-id path: the v2 small instance holds 1 536 rows (LsSmem<1536> fits the 48 KB of the
     // carry layout, so both run 4 blocks per SM); larger buckets go to the large instance
-    constexpr int kRowCap = (kPairs && kMin == 0 && kLsCap == 2048) ? 1536 : kLsCap;
+    constexpr int kRowCap = (kPairs && kMin == 0) ? 1024 : kLsCap;
     LsSmem<kRowCap> &S = *reinterpret_cast<LsSmem<kRowCap> *>(smem_raw);
     const int shift = plan->shift;
     const Q18SortSpec sp = plan->spec;
@@ -765,18 +766,18 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
         } else {
             // sub-bucket bits: ~8 rows per sub-bucket, at most kLsSubMax sub-buckets
             int sb = 0;
-            while (sb < 10 && (m >> (sb + 3)) > 0) ++sb;
+            while (sb < 9 && (m >> (sb + 3)) > 0) ++sb;
             if (sb > shift) sb = shift;
             const int ssh = shift - sb;
             const unsigned int ns = 1u << sb, smask = ns - 1u;
-            for (unsigned int i = threadIdx.x; i < ns; i += kBkThreads) S.sub[i] = 0;
+            for (unsigned int i = threadIdx.x; i < ns; i += kEmThreads) S.sub[i] = 0;
             __syncthreads();
-            for (unsigned int i0 = threadIdx.x; i0 < m; i0 += 2 * kBkThreads) {  // 2 loads in flight
+            for (unsigned int i0 = threadIdx.x; i0 < m; i0 += 2 * kEmThreads) {  // 2 loads in flight
                 unsigned long long kk[2];
                 unsigned int vv[2];
 #pragma unroll
                 for (int u = 0; u < 2; ++u) {
-                    const unsigned int i = i0 + u * kBkThreads;
+                    const unsigned int i = i0 + u * kEmThreads;
                     if (i < m) {
                         if (kPairs) {
                             const ulonglong2 kv = __ldcs(reinterpret_cast<const ulonglong2 *>(k) + lo + i);
@@ -790,7 +791,7 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
                 }
 #pragma unroll
                 for (int u = 0; u < 2; ++u) {
-                    const unsigned int i = i0 + u * kBkThreads;
+                    const unsigned int i = i0 + u * kEmThreads;
                     if (i >= m) break;
                     S.k1[i] = kk[u];
                     S.v1[i] = vv[u];
@@ -823,17 +824,17 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
                     if (i < ns) { S.sub[i] = run; S.cur[i] = run; }
                     run += c[q];
                 }
-                if (threadIdx.x == kBkThreads - 1) S.sub[ns] = run;
+                if (threadIdx.x == kEmThreads - 1) S.sub[ns] = run;
             }
             __syncthreads();
-            for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
+            for (unsigned int i = threadIdx.x; i < m; i += kEmThreads) {
                 const unsigned long long kk = S.k1[i];
                 const unsigned int p = atomicAdd(&S.cur[(unsigned int)(kk >> ssh) & smask], 1u);
                 S.k2[p] = kk;
                 S.v2[p] = S.v1[i];
             }
             __syncthreads();
-            for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {  // rank -> sorted smem
+            for (unsigned int i = threadIdx.x; i < m; i += kEmThreads) {  // rank -> sorted smem
                 const unsigned long long kk = S.k2[i];
                 const unsigned int sbk = (unsigned int)(kk >> ssh) & smask;
                 const unsigned int s0 = S.sub[sbk], s1 = S.sub[sbk + 1];
@@ -847,7 +848,7 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
             }
             __syncthreads();
             if (tiefix) {  // runs of equal 64-bit prefixes never cross buckets
-                for (unsigned int i = threadIdx.x; i < m; i += kBkThreads) {
+                for (unsigned int i = threadIdx.x; i < m; i += kEmThreads) {
                     const unsigned long long ki = S.k1[i];
                     if (i > 0 && S.k1[i - 1] == ki) continue;          // not a run head
                     if (i + 1 >= m || S.k1[i + 1] != ki) continue;     // run of one
@@ -870,11 +871,11 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
             }
         }
         __syncthreads();
-        for (unsigned int i0 = threadIdx.x; i0 < m; i0 += 2 * kBkThreads) {  // emit: 2 gathers in flight
+        for (unsigned int i0 = threadIdx.x; i0 < m; i0 += 2 * kEmThreads) {  // emit: 2 gathers in flight
             Q18Row row[2];
 #pragma unroll
             for (int u = 0; u < 2; ++u) {
-                const unsigned int i = i0 + u * kBkThreads;
+                const unsigned int i = i0 + u * kEmThreads;
                 if (i < m) {
                     const unsigned int r = S.v1[i];
                     unsigned long long *w64 = reinterpret_cast<unsigned long long *>(&row[u]);
@@ -884,7 +885,7 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
             }
 #pragma unroll
             for (int u = 0; u < 2; ++u) {
-                const unsigned int i = i0 + u * kBkThreads;
+                const unsigned int i = i0 + u * kEmThreads;
                 if (i >= m) break;
                 const unsigned long long a = sp.bits_a ? (S.k1[i] >> ashift) : 0ull;
                 const uint64_t j = lo + i;
@@ -919,10 +920,10 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
 // scattered 40 B/row writes cost more than the random gather they save) and sorting chunks of
 // whole buckets per block (fewer barriers, but 2 blocks/SM left the gathers latency-bound).
 constexpr int kObThreads = 1024;   // hist / scatter: 2 blocks of 32 warps per SM
-constexpr int kObCap = kLsCapSmall;  // per-bucket sort capacity: 2 048 rows (56 KB, 3 blocks/SM);
+constexpr int kObCap = 1536;  // per-bucket sort capacity (carry: 35 KB, 6 blocks of 128 threads/SM);
                                      // 4 096 (2 blocks/SM) with ~730-row buckets measured slower
 // dynamic shared memory of the v2 emit instances: row-id or carry layout, whichever is larger
-constexpr size_t kObSmem = sizeof(LsSmem<1536>) > sizeof(LcSmem<kObCap>) ? sizeof(LsSmem<1536>)
+constexpr size_t kObSmem = sizeof(LsSmem<1024>) > sizeof(LcSmem<kObCap>) ? sizeof(LsSmem<1024>)
                                                                          : sizeof(LcSmem<kObCap>);
 constexpr size_t kObSmemLarge = sizeof(LsSmem<kLsCapLarge>) > sizeof(LcSmem<kLcCapLarge>)
                                     ? sizeof(LsSmem<kLsCapLarge>) : sizeof(LcSmem<kLcCapLarge>);
@@ -1135,13 +1136,13 @@ void q18_bucket_order(const Q18Row *rows, const long long *amt, const Q18Plan *p
     end();
     begin("q18_bucket_sort_emit");
     unsigned lb = (unsigned)nb < (unsigned)num_sms * 3 ? (unsigned)nb : (unsigned)num_sms * 3;
-    bucket_local_emit_kernel<kLsCapSmall, 0><<<lb, kBkThreads, sizeof(LsSmem<kLsCapSmall>), st>>>(
+    bucket_local_emit_kernel<kLsCapSmall, 0><<<lb, kEmThreads, sizeof(LsSmem<kLsCapSmall>), st>>>(
         s.k[1], s.v[1], s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
     end();
     // buckets above the small capacity (skewed keys): one block per SM, ~200 KB shared memory
     begin("q18_bucket_sort_emit_large");
-    bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall><<<(unsigned)num_sms, kBkThreads,
+    bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall><<<(unsigned)num_sms, kEmThreads,
                                                           sizeof(LsSmem<kLsCapLarge>), st>>>(
         s.k[1], s.v[1], s.offset, nb, plan, rows, amt, dst, flag, s.big);
     count_launches(1);
@@ -1206,13 +1207,13 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
     end();
     // per-bucket shared-memory sort + tie-fix + emit: the v1 kernels on the (key, row id) pairs
     begin("q18_bucket_sort_emit");
-    const unsigned lb = (unsigned)nb < (unsigned)num_sms * 4 ? (unsigned)nb : (unsigned)num_sms * 4;
-    launch_pdl(bucket_local_emit_kernel<kObCap, 0, true>, lb, kBkThreads, kObSmem, st,
+    const unsigned lb = (unsigned)nb < (unsigned)num_sms * 6 ? (unsigned)nb : (unsigned)num_sms * 6;
+    launch_pdl(bucket_local_emit_kernel<kObCap, 0, true>, lb, kEmThreads, kObSmem, st,
         s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2);
     count_launches(1);
     end();
     begin("q18_bucket_sort_emit_large");
-    launch_pdl(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>, (unsigned)num_sms, kBkThreads, kObSmemLarge, st,
+    launch_pdl(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>, (unsigned)num_sms, kEmThreads, kObSmemLarge, st,
         s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2);
     count_launches(1);
     end();
