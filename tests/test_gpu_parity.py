@@ -623,3 +623,33 @@ def test_full_size_w100_strict(h):
         assert_q18(L.q(18), oracle.q18(t, Q18_HAVING))
     finally:
         h.h2tap_close(e)
+
+
+def test_full_size_w1000_q6_q1_shared_batch(h):
+    """Config C4 size on one GPU: W=1000 (~300 M order_line rows, 7.2 GB of Q1/Q6 columns),
+    Q6 + Q1 as one batch (the shared scan) and separately, vs the oracle on every row."""
+    cols = ["ol_number", "ol_delivery_d", "ol_quantity", "ol_amount"]
+    parts = []
+    for lo in range(1, 1001, 50):
+        g = chgen.generate(lo, lo + 50, seed=1, with_item=False)
+        parts.append({c: g["order_line"][c] for c in cols})
+    ol = {c: np.concatenate([p[c] for p in parts]) for c in cols}
+    del parts
+    t = {"order_line": ol}
+    want6 = oracle.q6(t, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI)
+    want1 = oracle.q1(t, Q1_CUTOFF)
+    e = h.h2tap_open(0)
+    try:
+        h.h2tap_load_snapshot(e, t, 1)
+        rs = h.h2tap_run_queries(e, [(6, None, 0), (1, None, 0)])
+        g6, g1 = rs[0].to_numpy(), rs[1].to_numpy()
+        g6["_nulls"] = dict(rs[0].nulls)
+        for r in rs:
+            h.h2tap_free(r)
+        assert_q6(g6, want6)
+        assert_q1(g1, want1)
+        L = Loader(h, e)
+        assert_q6(L.q(6), want6)
+        assert_q1(L.q(1), want1)
+    finally:
+        h.h2tap_close(e)
