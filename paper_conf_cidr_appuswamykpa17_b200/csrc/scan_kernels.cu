@@ -472,9 +472,9 @@ template <int kS> struct Q1StagesT {
 // Q1 alone: 8 aggregating warps, 5 stages (208 KB). Shared with Q6: 12 aggregating warps (their
 // latency-bound slot updates were the shared pass's limit) and 4 stages (224 KB).
 template <bool kQ6> struct Q1TmaCfg {
-    static constexpr int kW = kQ6 ? 12 : kTmaConsumerWarps;  // aggregating warps
+    static constexpr int kW = 12;                             // aggregating warps
     static constexpr int kT = kW * 32;
-    static constexpr int kS = kQ6 ? 4 : 5;                    // ring stages
+    static constexpr int kS = 4;                              // ring stages
 };
 
 // kQ6: shared scan of a batch's Q6 and Q1 — Q6 reads a subset of Q1's columns
@@ -487,7 +487,7 @@ template <bool kQ6> struct Q1TmaCfg {
 constexpr int kQ6SideWarps = 4;
 constexpr int kQ61Threads = (Q1TmaCfg<true>::kW + 1 + kQ6SideWarps) * 32;
 template <bool kQ6>
-__global__ void __launch_bounds__(kQ6 ? kQ61Threads : kTmaThreads, 1)
+__global__ void __launch_bounds__(kQ6 ? kQ61Threads : (Q1TmaCfg<false>::kW + 1) * 32, 1)
 q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deliv,
               const int *__restrict__ qty, const long long *__restrict__ amt, uint64_t n,
               long long cutoff, Q1Scratch g, Q6Pred pred6, long long *__restrict__ part6,
@@ -807,7 +807,7 @@ void launch_q1_tma(const int32_t *number, const int64_t *deliv, const int32_t *q
     }
     const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
     const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
-    launch_pdl(q1_tma_kernel<false>, grid, kTmaThreads, smem, st, number, reinterpret_cast<const long long *>(deliv), qty,
+    launch_pdl(q1_tma_kernel<false>, grid, (Q1TmaCfg<false>::kW + 1) * 32, smem, st, number, reinterpret_cast<const long long *>(deliv), qty,
                reinterpret_cast<const long long *>(amt), n, cutoff, s, Q6Pred{0, 0, 0, 0}, nullptr, nullptr,
                nullptr, nullptr);
     count_launches(1);
