@@ -484,7 +484,7 @@ template <bool kQ6> struct Q1TmaCfg {
 // Shared-scan block: warps 0-7 Q1 (as above), warp 8 the producer, warps 9-12 Q6 on the same
 // staged chunks (registers only) — Q6 added to the Q1 warps' rows lengthened their dependent
 // shared-memory update chains (145 vs 117 us); separate warps run it alongside.
-constexpr int kQ6SideWarps = 4;
+constexpr int kQ6SideWarps = 6;
 constexpr int kQ61Threads = (Q1TmaCfg<true>::kW + 1 + kQ6SideWarps) * 32;
 template <bool kQ6>
 __global__ void __launch_bounds__(kQ6 ? kQ61Threads : (Q1TmaCfg<false>::kW + 1) * 32, 1)
@@ -557,9 +557,12 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
             const unsigned rows = (unsigned)(n - c * kQ1Chunk < (uint64_t)kQ1Chunk ? n - c * kQ1Chunk
                                                                                  : (uint64_t)kQ1Chunk);
             if (rows == (unsigned)kQ1Chunk) {  // full chunk: 128-bit / 64-bit shared loads of pairs
+                constexpr int kPairs = kQ1Chunk / 2, kStep = kQ6SideWarps * 32;
+                static_assert(kPairs % kStep == 0 || kQ6SideWarps != 4, "full-chunk pair loop");
 #pragma unroll
-                for (int k = 0; k < kQ1Chunk / (2 * kQ6SideWarps * 32); ++k) {
-                    const unsigned pr = t6 + k * kQ6SideWarps * 32;
+                for (int k = 0; k < (kPairs + kStep - 1) / kStep; ++k) {
+                    const unsigned pr = t6 + k * kStep;
+                    if (kPairs % kStep != 0 && pr >= (unsigned)kPairs) break;
                     const longlong2 d2 = reinterpret_cast<const longlong2 *>(P.deliv[s])[pr];
                     const longlong2 a2 = reinterpret_cast<const longlong2 *>(P.amt[s])[pr];
                     const int2 q2 = reinterpret_cast<const int2 *>(P.qty[s])[pr];
