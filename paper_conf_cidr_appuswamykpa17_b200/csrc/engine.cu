@@ -519,6 +519,19 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
     std::lock_guard<std::mutex> g(e->load_mu);
     CK(cudaSetDevice(e->device));
     publish_ready(e, false);
+    // back-pressure: at most 3 refreshes in flight (each may hold a snapshot copy), so a stream
+    // of async loads reaches a steady state the memory pool can serve without growing
+    // (polled: a query thread may publish — and release — the oldest refresh concurrently)
+    for (;;) {
+        size_t inflight;
+        {
+            std::lock_guard<std::mutex> gp(e->pend_mu);
+            inflight = e->pending.size();
+        }
+        if (inflight < 3) break;
+        std::this_thread::sleep_for(std::chrono::microseconds(50));
+        publish_ready(e, false);
+    }
     if (e->any_epoch && epoch <= e->last_epoch.load())
         return fail(H2TAP_ESTALE, "epoch %llu is not greater than the last accepted epoch %llu",
                     (unsigned long long)epoch, (unsigned long long)e->last_epoch.load());
