@@ -458,9 +458,10 @@ q1_kernel(const int4 *__restrict__ number, const longlong2 *__restrict__ deliv,
     q1_block_merge(sm, g, tid);
 }
 
-// Q1, TMA-bulk pipelined variant: one block per SM, warp 8 streams 1024-row chunks of the four
-// columns into a 4-stage ring (96 KB) next to the 88 KB of aggregation tables; warps 0-7
-// aggregate exactly as q1_kernel does (thread-private dense slots, warp-aggregated sparse path).
+// Q1, TMA-bulk pipelined variant: one block per SM; the producer warp streams 1024-row chunks of
+// the four columns into a 4-stage ring (96 KB) next to 12 aggregating warps' slot tables
+// (120 KB): thread-private dense slots, warp-aggregated sparse path (as q1_kernel). 12 warps
+// instead of 8: the slot updates are latency-bound.
 constexpr int kQ1Chunk = 1024;
 template <int kS> struct Q1StagesT {
     long long deliv[kS][kQ1Chunk];

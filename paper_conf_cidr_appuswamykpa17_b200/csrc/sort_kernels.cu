@@ -5,8 +5,10 @@
 // min/max (HAVING kernel statistics) and the snapshot's zone maps: a = max - amount_sum (DESC),
 // e = o_entry_d - min, r = (w, d, o) offsets as concatenated fixed-width fields. a|e|r is the
 // exact composite key.
-//  * main path: sort (top 64 bits of a|e|r, row id) pairs with a bucket sort (partition by the
-//    top key bits, bitonic sort per bucket in shared memory). If a|e|r fits 64 bits the keys are
+//  * main path: a bucket sort (partition by the top key bits, then a sub-bucket partition and
+//    rank counting per bucket in shared memory) of 128-bit carry records that hold the whole
+//    result row when it fits, else of (top 64 bits of a|e|r, row id) pairs.
+//    For the pairs: if a|e|r fits 64 bits the keys are
 //    distinct and the order is exact; otherwise runs of equal 64-bit prefixes are ordered by the
 //    full tuple (tie-fix; runs are a handful of rows on realistic data).
 //  * exact fallback (a run > 32 rows or a bucket > shared memory): one stable LSD radix sort of
@@ -419,7 +421,7 @@ namespace {
 
 constexpr int kBkThreads = 256;
 constexpr int kBkItems = 16;                       // rows per thread in the scatter
-constexpr int kLsCapSmall = 2048;                  // rows per bucket: fast kernel (3 blocks/SM)
+constexpr int kLsCapSmall = 2048;                  // rows per bucket: v1 small instance
 constexpr int kLsCapLarge = 8192;                  // rows per bucket: large-bucket kernel
 constexpr int kLsSubMax = 512;                     // max sub-buckets per bucket (4 per emit thread)
 constexpr int kEmThreads = 128;                    // per-bucket sort / emit block (8 blocks/SM)
@@ -543,9 +545,8 @@ template <int kLsCap> struct LsSmem {
     unsigned int wsum[kEmThreads / 32];
 };
 
-// carry mode: 64-bit second words instead of 32-bit row ids (2 048 rows: 72 KB, 3 blocks/SM)
-// (records stay where they were loaded; the sort moves 16-bit indices: 48 KB for 2 048 rows,
-// 4 blocks per SM)
+// carry mode: the records stay where they were loaded and the sort moves 16-bit record ids
+// (1 536 rows: 35 KB, 6 blocks of 128 threads per SM)
 template <int kCap> struct LcSmem {
     ulonglong2 rec[kCap];             // the bucket's records, load order
     unsigned short idx[kCap];         // record ids grouped by sub-bucket
