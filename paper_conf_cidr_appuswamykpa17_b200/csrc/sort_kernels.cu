@@ -737,8 +737,8 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
             reinterpret_cast<const ulonglong2 *>(k), offset, nb, plan, dst, flag, big, smem_raw, sub_log2);
         return;
     }
-    // row-id path: the v2 small instance holds 1 536 rows (LsSmem<1536> fits the 48 KB of the
-    // carry layout, so both run 4 blocks per SM); larger buckets go to the large instance
+    // row-id path: the v2 small instance holds 1 024 rows (LsSmem<1024> fits the 35 KB of the
+    // carry layout, so both run 6 blocks per SM); larger buckets go to the large instance
     constexpr int kRowCap = (kPairs && kMin == 0) ? 1024 : kLsCap;
     LsSmem<kRowCap> &S = *reinterpret_cast<LsSmem<kRowCap> *>(smem_raw);
     const int shift = plan->shift;
