@@ -1120,9 +1120,10 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     // carry records unless disabled for A/B (H2TAP_ORDER_CARRY=0) or on v1
     const char *cv = std::getenv("H2TAP_ORDER_CARRY");
     const bool carry = !e->order_v1 && !(cv && cv[0] == '0');
-    e->prof.run("q18_plan", [&] {
-        launch_q18_plan(q.q18.stats, q.zone, q.q18.nout, bb, carry, q.plan_dev, q.q18.tie, e->compute);
-    });
+    if (e->order_v1)  // (the v2 histogram kernel derives the plan itself)
+        e->prof.run("q18_plan", [&] {
+            launch_q18_plan(q.q18.stats, q.zone, q.q18.nout, bb, carry, q.plan_dev, q.q18.tie, e->compute);
+        });
     for (int b = 0; b < 2; ++b) {
         q.sp.k[b] = static_cast<unsigned long long *>(e->arena.get("q18.sk" + std::to_string(b), 8 * n_max));
         q.sp.v[b] = static_cast<unsigned int *>(e->arena.get("q18.sv" + std::to_string(b), 4 * n_max));
@@ -1170,8 +1171,9 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     } else {
         bs.mat = static_cast<unsigned int *>(e->arena.get("q18.bmat", 4ull * ob_grid(e->num_sms) << kBucketMaxBits));
         bs.kv = static_cast<unsigned long long *>(e->arena.get("q18.kv", 16 * n_max));
+        const Q18PlanArgs pa{q.q18.stats, q.zone, q.q18.nout, carry ? 1 : 0};
         q18_bucket_order_v2(q.rows, q.amt, q.plan_dev, n_max, bb, bs, d, q.tie_dev, e->num_sms, e->compute,
-                            &marks);
+                            &marks, &pa);
     }
 }
 

@@ -225,9 +225,17 @@ void q18_bucket_order(const Q18Row *rows, const long long *amt, const Q18Plan *p
 // column scan), keys computed in the scatter; the per-bucket sort + emit kernels are v1's.
 int ob_grid(int num_sms);
 int ob_bucket_bits(uint64_t n_max);
-void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan *plan, uint64_t n_max,
+// The inputs of the ORDER BY plan when the v2 histogram kernel computes it (no plan launch).
+struct Q18PlanArgs {
+    const Q18Stats *stats;
+    Q18Zone zone;
+    const unsigned long long *nout;
+    int allow_carry;
+};
+void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, Q18Plan *plan, uint64_t n_max,
                          int bucket_bits, const BucketSort &s, const Q18Cols &dst, unsigned int *flag,
-                         int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr);
+                         int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr,
+                         const Q18PlanArgs *plan_args = nullptr);  // non-null: hist writes *plan
 // Within runs of equal prefix, order by the full tuple; runs longer than 32 raise *flag.
 // Exact fallback: three stable passes over the full fields (row rank, entry, amount).
 void launch_q18_field_keys(const Q18Row *rows, const long long *amt, const unsigned int *vals,

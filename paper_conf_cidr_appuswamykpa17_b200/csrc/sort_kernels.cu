@@ -312,14 +312,9 @@ __global__ void permute_kernel(const Q18Row *__restrict__ rows, const long long 
 
 __device__ __forceinline__ int bitwidth_dev(unsigned long long x) { return x ? 64 - __clzll(x) : 0; }
 
-// One thread: the ORDER BY plan from the HAVING statistics (amount_sum, o_entry_d) and the
-// snapshot's zone maps (w, d, o; carry payload): widths of a, e, r, the prefix width, and
-// whether the 128-bit carry record holds the whole row.
-__global__ void q18_plan_kernel(const Q18Stats *__restrict__ stats, Q18Zone z,
-                                const unsigned long long *nout, int bucket_bits, int allow_carry,
-                                Q18Plan *plan, unsigned int *flag) {
-    pdl_wait();
-    pdl_trigger();
+__device__ Q18Plan make_q18_plan(const Q18Stats *__restrict__ stats, const Q18Zone &z,
+                                 const unsigned long long *nout, int bucket_bits, int allow_carry,
+                                 unsigned int *flag) {
     const Q18Stats st = *stats;
     Q18Plan p{};
     p.n = *nout;
@@ -335,7 +330,7 @@ __global__ void q18_plan_kernel(const Q18Stats *__restrict__ stats, Q18Zone z,
         sp.bits_e = bitwidth_dev((unsigned long long)st.ent_max - (unsigned long long)st.ent_min);
         // (the join-key domain, w < 2^23, d < 2^8, o >= 0, keeps this <= 62; guard anyway)
         sp.wide_r = sp.bits_w + sp.bits_d + sp.bits_o > 62;
-        if (sp.wide_r) atomicOr(flag, 4u);  // the engine redoes the ORDER BY per column
+        if (sp.wide_r && flag) atomicOr(flag, 4u);  // the engine redoes the ORDER BY per column
         sp.bits_r = sp.wide_r ? 62 : sp.bits_w + sp.bits_d + sp.bits_o;
         const int B = sp.bits_a + sp.bits_e + sp.bits_r;
         sp.prefix_bits = B <= 64 ? B : 64;
@@ -348,7 +343,19 @@ __global__ void q18_plan_kernel(const Q18Stats *__restrict__ stats, Q18Zone z,
         p.tiefix = B > 64 && !sp.carry;  // carry records compare all key bits: no tie-fix
         p.shift = sp.prefix_bits > bucket_bits ? sp.prefix_bits - bucket_bits : 0;
     }
-    *plan = p;
+    return p;
+}
+
+// One thread: the ORDER BY plan from the HAVING statistics (amount_sum, o_entry_d) and the
+// snapshot's zone maps (w, d, o; carry payload): widths of a, e, r, the prefix width, and
+// whether the 128-bit carry record holds the whole row. (The v2 ORDER BY computes it inside
+// its histogram kernel instead: one launch less.)
+__global__ void q18_plan_kernel(const Q18Stats *__restrict__ stats, Q18Zone z,
+                                const unsigned long long *nout, int bucket_bits, int allow_carry,
+                                Q18Plan *plan, unsigned int *flag) {
+    pdl_wait();
+    pdl_trigger();
+    *plan = make_q18_plan(stats, z, nout, bucket_bits, allow_carry, flag);
 }
 
 unsigned grid_cap(uint64_t work, int threads, int num_sms, int per_sm) {
@@ -947,15 +954,27 @@ __device__ __forceinline__ void ob_range(uint64_t n, uint64_t &r0, uint64_t &r1)
 
 __global__ void __launch_bounds__(kObThreads)
 ob_hist_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
-               const Q18Plan *__restrict__ plan, int nb, unsigned int *__restrict__ mat,
-               unsigned int *__restrict__ big) {
+               Q18Plan *__restrict__ plan, int nb, unsigned int *__restrict__ mat,
+               unsigned int *__restrict__ big, int make_plan, Q18PlanArgs pa, int bucket_bits,
+               unsigned int *flag) {
     pdl_wait();
     pdl_trigger();
     extern __shared__ unsigned int h[];
+    __shared__ Q18Plan P;
     if (blockIdx.x == 0 && threadIdx.x == 0) *big = 0;  // work-list count of the emit kernels
-    const uint64_t n = plan->n;
-    const Q18SortSpec sp = plan->spec;
-    const int shift = plan->shift;
+    if (make_plan) {  // every block derives the plan (a few dozen instructions); block 0 stores it
+        if (threadIdx.x == 0) {
+            P = make_q18_plan(pa.stats, pa.zone, pa.nout, bucket_bits, pa.allow_carry,
+                              blockIdx.x == 0 ? flag : nullptr);
+            if (blockIdx.x == 0) *plan = P;
+        }
+    } else if (threadIdx.x == 0) {
+        P = *plan;
+    }
+    __syncthreads();
+    const uint64_t n = P.n;
+    const Q18SortSpec sp = P.spec;
+    const int shift = P.shift;
     const bool amt_only = sp.bits_a > 0 && shift >= sp.prefix_bits - sp.bits_a;
     for (int i = threadIdx.x; i < nb; i += kObThreads) h[i] = 0;
     __syncthreads();
@@ -1167,9 +1186,9 @@ int ob_bucket_bits(uint64_t n_max) {  // ~256-512 rows per bucket
     return bb;
 }
 
-void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan *plan, uint64_t n_max,
+void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, Q18Plan *plan, uint64_t n_max,
                          int bucket_bits, const BucketSort &s, const Q18Cols &dst, unsigned int *flag,
-                         int num_sms, cudaStream_t st, PhaseMarks *marks) {
+                         int num_sms, cudaStream_t st, PhaseMarks *marks, const Q18PlanArgs *plan_args) {
     auto begin = [&](const char *nm) { if (marks) marks->begin(nm); };
     auto end = [&] { if (marks) marks->end(); };
     if (bucket_bits > kBucketMaxBits) bucket_bits = kBucketMaxBits;
@@ -1194,7 +1213,9 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, const Q18Plan
         return v ? std::max(0, std::min(6, std::atoi(v))) : 1;  // measured: 1 -> 74 us, 3 -> 84 us
     }();
     begin("q18_sort_hist");
-    launch_pdl(ob_hist_kernel, G, kObThreads, nb * 4, st, rows, amt, plan, nb, s.mat, s.big);
+    const Q18PlanArgs pa = plan_args ? *plan_args : Q18PlanArgs{};
+    launch_pdl(ob_hist_kernel, G, kObThreads, nb * 4, st, rows, amt, plan, nb, s.mat, s.big,
+               plan_args ? 1 : 0, pa, bucket_bits, flag);
     count_launches(1);
     end();
     begin("q18_sort_scan");
