@@ -129,6 +129,15 @@ def _check(st):
         raise MemoryError("oracle out of memory")
 
 
+def ts_cmp(op: str, v, c):
+    """The oracle's 3-valued timestamp comparison (v is None = SQL NULL): True, False or None."""
+    lib = _load()
+    code = {">=": 0, "<": 1, ">": 2}[op]
+    vv = np.iinfo(np.int64).min if v is None else int(v)
+    r = lib.oracle_ts_cmp(C.c_int(code), C.c_int64(vv), C.c_int64(int(c)))
+    return {0: False, 1: True, 2: None}[r]
+
+
 def q6(tables, d_lo, d_hi, q_lo, q_hi):
     """CH Q6. Returns {"revenue": int or None (NULL), "count": qualifying rows}."""
     lib, keep = _load(), _Keep()

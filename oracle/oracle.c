@@ -38,6 +38,20 @@ static sqlbool between(int64_t x, int64_t lo, int64_t hi) {
     return sql_and(x >= lo ? SQL_TRUE : SQL_FALSE, x <= hi ? SQL_TRUE : SQL_FALSE);
 }
 
+/* Test hook (test infrastructure only): the timestamp comparisons above, exported so a test
+ * can pin their three-valued results against SQLite's NULL semantics, including a constant
+ * equal to the sentinel's own value (a NULL test dropped from one helper is otherwise masked
+ * in Q6, where ts_ge is ANDed with ts_lt's UNKNOWN). op: 0 = '>=', 1 = '<', 2 = '>'.
+ * Returns 0 FALSE, 1 TRUE, 2 UNKNOWN; -1 for an unknown op. */
+int oracle_ts_cmp(int op, int64_t v, int64_t c) {
+    switch (op) {
+        case 0: return (int)ts_ge(v, c);
+        case 1: return (int)ts_lt(v, c);
+        case 2: return (int)ts_gt(v, c);
+        default: return -1;
+    }
+}
+
 /* ------------------------------------------------------- generic hash map -- */
 /* Keys are tuples of k int64 values; each entry carries an int64 payload.
  * Used both as a multimap (join index: every row inserted) and as a map

@@ -67,6 +67,10 @@ typedef struct {
 #define OR_OVERFLOW -1   /* an int64 SUM overflowed (SQLite raises "integer overflow") */
 #define OR_NOMEM    -2
 
+/* 3-valued comparison of a (possibly NULL = INT64_MIN) timestamp v with constant c, as the
+ * queries below evaluate it; op 0 '>=', 1 '<', 2 '>'. Returns 0 FALSE, 1 TRUE, 2 UNKNOWN. */
+int oracle_ts_cmp(int op, int64_t v, int64_t c);
+
 /* CH Q6: SELECT SUM(ol_amount) FROM order_line WHERE ol_delivery_d >= d_lo AND
  * ol_delivery_d < d_hi AND ol_quantity BETWEEN q_lo AND q_hi.
  * *revenue_is_null = 1 when no row qualifies (SUM over the empty set is NULL).

@@ -28,6 +28,11 @@ def iso_us(s: str) -> int:
     return (int(t.replace(microsecond=0).timestamp()) * 1_000_000) + t.microsecond
 
 
+def ts_param(v) -> int:
+    """A fixture parameter: an ISO timestamp string (-> int64 µs UTC) or a raw int64."""
+    return iso_us(v) if isinstance(v, str) else int(v)
+
+
 # CH-benCHmark literal constants, converted independently of the oracle and the library.
 Q1_CUTOFF = iso_us("2007-01-02T00:00:00")
 Q6_D_LO = iso_us("1999-01-01T00:00:00")

@@ -13,7 +13,8 @@ import pytest
 
 import chgen
 import oracle
-from chref import (Q1_CUTOFF, Q6_D_HI, Q6_D_LO, Q6_Q_HI, Q6_Q_LO, Q18_HAVING, golden, iso_us)
+from chref import (Q1_CUTOFF, Q6_D_HI, Q6_D_LO, Q6_Q_HI, Q6_Q_LO, Q18_HAVING, golden, iso_us,
+                   ts_param)
 
 pytestmark = pytest.mark.gpu
 HASH = 4  # H2TAP_QUERY_HASH_JOIN
@@ -137,6 +138,45 @@ def test_golden_fixture(L):
         assert got["amount_sum"].tolist() == [r["amount_sum"] for r in case["rows"]]
         assert got["o_entry_d"].tolist() == [iso_us(r["o_entry_d"]) for r in case["rows"]]
         assert got["c_last"].tolist() == [r["c_last"] for r in case["rows"]]
+
+
+def test_boundaries_fixture(L, order_mode):
+    """tests/golden/boundaries_ch.json: rows exactly on every predicate bound (Q6 d_lo/d_hi, BETWEEN
+    ends, Q1 cutoff, NULL vs INT64_MIN constants) and a Q18 group summing to exactly the HAVING
+    threshold; hand-derived expectations (also pinned by SQLite and brute force on the CPU)."""
+    t, exp = golden("boundaries_ch.json")
+    L.load(t)
+    for case in exp["q6"]:
+        p = [ts_param(v) for v in case["params"]]
+        assert_q6(L.q(6, p), {"revenue": case["revenue"], "count": case["count"]})
+    for case in exp["q1"]:
+        got = L.q(1, [ts_param(case["params"][0])])
+        rows = case["rows"]
+        for k in ("ol_number", "sum_qty", "sum_amount", "count_order"):
+            assert got[k].tolist() == [r[k] for r in rows], (case["_why"], k)
+        for k in ("avg_qty", "avg_amount"):
+            for a, b in zip(got[k].tolist(), [r[k] for r in rows]):
+                assert math.isclose(a, b, rel_tol=1e-9, abs_tol=0.0), (case["_why"], k)
+    for case in exp["q18"]:
+        for flags in (0, HASH):
+            got = L.q(18, case["params"], flags=flags)
+            want = [(r["c_last"], r["c_id"], r["o_id"], iso_us(r["o_entry_d"]), r["o_ol_cnt"],
+                     r["amount_sum"], r["o_w_id"], r["o_d_id"]) for r in case["rows"]]
+            assert list(zip(*[got[k].tolist() for k in Q18_NAMES])) == want, case["_why"]
+
+
+def test_q18_having_exactly_at_group_sums(L, order_mode):
+    """HAVING thresholds equal to existing group sums (the '>' boundary) at W=2: the group at the
+    threshold is excluded, the one 1 cent above it included, on both join-index layouts."""
+    t = chgen.generate(1, 3, seed=21)
+    L.load(t)
+    sums = oracle.q18(t, -1)["amount_sum"]
+    picks = sorted({int(sums[0]), int(sums[len(sums) // 2]), int(sums[-1]), Q18_HAVING})
+    for thr in picks + [picks[1] - 1, picks[1] + 1]:
+        want = oracle.q18(t, thr)
+        assert thr not in want["amount_sum"].tolist()
+        assert_q18(L.q(18, [thr]), want)
+        assert_q18(L.q(18, [thr], flags=HASH), want)
 
 
 @pytest.mark.parametrize("W,mode,seed", [(1, "spread", 1), (3, "spread", 2), (2, "strict", 3)])
