@@ -2,13 +2,15 @@
 
 Thin Python binding of the C ABI in ``include/h2tap.h`` (``libh2tap.so``, built in-tree by
 ``_build.py`` for sm_100a). Every function here only marshals arguments: the snapshot store,
-the query kernels, the NCCL merge and the finalisation all run in the CUDA library. There is
+the query kernels, the cross-GPU merge (peer-memory kernels) and the finalisation all run in
+the CUDA library. There is
 no CPU fallback — importing this package fails loudly when the library is missing.
 
 Names mirror the ABI: ``h2tap_open``, ``h2tap_load_snapshot``, ``h2tap_sync``,
 ``h2tap_refresh``, ``h2tap_refresh_rows``, ``h2tap_get_store_stats``,
 ``h2tap_run_query``, ``h2tap_free``, ``h2tap_close``, ``h2tap_last_error``,
-``h2tap_nccl_unique_id``, ``h2tap_compute_stream``, ``h2tap_c_last_name``.
+``h2tap_peer_handle``, ``h2tap_peer_connect``, ``h2tap_peer_connect_local``,
+``h2tap_compute_stream``, ``h2tap_c_last_name``.
 """
 from __future__ import annotations
 
@@ -29,8 +31,8 @@ _lib = C.CDLL(LIB_PATH)
 
 # ------------------------------------------------------------------ ABI types --
 H2TAP_OK, H2TAP_EINVAL, H2TAP_ESTALE, H2TAP_ENOMEM = 0, -1, -2, -3
-H2TAP_ECUDA, H2TAP_ENCCL, H2TAP_EPLAN, H2TAP_EDUPKEY, H2TAP_ESHAPE = -4, -5, -6, -7, -8
-STATUS_NAMES = {0: "OK", -1: "EINVAL", -2: "ESTALE", -3: "ENOMEM", -4: "ECUDA", -5: "ENCCL",
+H2TAP_ECUDA, H2TAP_EPEER, H2TAP_EPLAN, H2TAP_EDUPKEY, H2TAP_ESHAPE = -4, -5, -6, -7, -8
+STATUS_NAMES = {0: "OK", -1: "EINVAL", -2: "ESTALE", -3: "ENOMEM", -4: "ECUDA", -5: "EPEER",
                 -6: "EPLAN", -7: "EDUPKEY", -8: "ESHAPE", -9: "EOVERFLOW"}
 H2TAP_I32, H2TAP_I64, H2TAP_F64 = 1, 2, 3
 H2TAP_T_ORDER_LINE, H2TAP_T_ORDERS, H2TAP_T_CUSTOMER, H2TAP_T_ITEM, H2TAP_T_NEW_ORDER = 1, 2, 3, 4, 5
@@ -99,7 +101,7 @@ class h2tap_store_stats(C.Structure):
 
 class h2tap_config(C.Structure):
     _fields_ = [("device", C.c_int), ("rank", C.c_int), ("world", C.c_int),
-                ("nccl_unique_id", C.c_void_p)]
+                ("peer_heap_bytes", C.c_uint64)]
 
 
 class h2tap_query(C.Structure):
@@ -114,7 +116,8 @@ class h2tap_result(C.Structure):
                 ("nulls", C.POINTER(C.POINTER(C.c_uint8))), ("rows_scanned", C.c_uint64),
                 ("device_ms", C.c_double), ("e2e_ms", C.c_double), ("nkernels", C.c_uint32),
                 ("kernel_names", C.POINTER(C.c_char_p)), ("kernel_ms", C.POINTER(C.c_double)),
-                ("kernel_launches", C.c_uint64), ("plan_flags", C.c_uint32)]
+                ("kernel_launches", C.c_uint64), ("plan_flags", C.c_uint32),
+                ("row_offset", C.c_uint64), ("total_rows", C.c_uint64)]
 
 
 class h2tap_layout_table(C.Structure):
@@ -148,21 +151,24 @@ _lib.h2tap_free.restype = None
 _lib.h2tap_close.argtypes = [_P]
 _lib.h2tap_close.restype = None
 _lib.h2tap_last_error.restype = C.c_char_p
-_lib.h2tap_nccl_unique_id.argtypes = [_P]
+_lib.h2tap_peer_handle.argtypes = [_P, _P]
+_lib.h2tap_peer_connect.argtypes = [_P, _P, C.c_uint32]
+_lib.h2tap_peer_connect_local.argtypes = [C.POINTER(_P), C.c_uint32]
 _lib.h2tap_compute_stream.argtypes = [_P, C.POINTER(_P)]
 _lib.h2tap_c_last_name.argtypes = [C.c_int32, C.c_char_p, C.c_size_t]
 for _f in ("h2tap_open", "h2tap_load_snapshot_ex", "h2tap_load_snapshot", "h2tap_load_snapshot_rows",
            "h2tap_reserve", "h2tap_refresh", "h2tap_refresh_rows", "h2tap_get_store_stats",
            "h2tap_sync",
-           "h2tap_run_query_ex", "h2tap_run_query", "h2tap_run_queries", "h2tap_nccl_unique_id",
-           "h2tap_compute_stream", "h2tap_layout_sum"):
+           "h2tap_run_query_ex", "h2tap_run_query", "h2tap_run_queries", "h2tap_peer_handle",
+           "h2tap_peer_connect", "h2tap_peer_connect_local", "h2tap_compute_stream", "h2tap_layout_sum"):
     getattr(_lib, _f).restype = C.c_int
 
 ABI_SYMBOLS = ["h2tap_open", "h2tap_load_snapshot", "h2tap_load_snapshot_ex",
                "h2tap_load_snapshot_rows", "h2tap_reserve", "h2tap_refresh", "h2tap_refresh_rows",
                "h2tap_get_store_stats", "h2tap_sync",
                "h2tap_run_query", "h2tap_run_query_ex", "h2tap_run_queries", "h2tap_free", "h2tap_close",
-               "h2tap_last_error", "h2tap_nccl_unique_id", "h2tap_compute_stream",
+               "h2tap_last_error", "h2tap_peer_handle", "h2tap_peer_connect",
+               "h2tap_peer_connect_local", "h2tap_compute_stream",
                "h2tap_c_last_name", "h2tap_layout_sum"]
 
 
@@ -195,18 +201,77 @@ class Engine:
         h2tap_close(self)
 
 
-def h2tap_nccl_unique_id() -> bytes:
-    buf = C.create_string_buffer(128)
-    _check(_lib.h2tap_nccl_unique_id(C.cast(buf, _P)))
-    return buf.raw
-
-
-def h2tap_open(device: int = 0, rank: int = 0, world: int = 1, nccl_unique_id: bytes | None = None) -> Engine:
-    idbuf = C.create_string_buffer(nccl_unique_id, 128) if nccl_unique_id is not None else None
-    cfg = h2tap_config(device, rank, world, C.cast(idbuf, _P) if idbuf is not None else None)
+def h2tap_open(device: int = 0, rank: int = 0, world: int = 1, peer_heap_bytes: int = 0) -> Engine:
+    cfg = h2tap_config(device, rank, world, peer_heap_bytes)
     h = _P()
     _check(_lib.h2tap_open(C.byref(cfg), C.byref(h)))
     return Engine(h, device, rank, world)
+
+
+def h2tap_peer_handle(engine: Engine) -> bytes:
+    """This rank's 64-byte CUDA IPC handle of its peer segment (world > 1)."""
+    buf = C.create_string_buffer(64)
+    _check(_lib.h2tap_peer_handle(engine.handle, C.cast(buf, _P)))
+    return buf.raw
+
+
+def h2tap_peer_connect(engine: Engine, handles) -> None:
+    """Map every rank's peer segment (``handles``: the world's 64-byte handles in rank order)."""
+    blob = b"".join(bytes(h) for h in handles)
+    buf = C.create_string_buffer(blob, len(blob))
+    _check(_lib.h2tap_peer_connect(engine.handle, C.cast(buf, _P), len(handles)))
+
+
+def h2tap_peer_connect_local(engines) -> None:
+    """Connect engines of ONE process (engines[k] has rank k); they may share a device."""
+    arr = (_P * len(engines))(*[e.handle for e in engines])
+    _check(_lib.h2tap_peer_connect_local(arr, len(engines)))
+
+
+def open_local_group(world: int, device: int = 0, peer_heap_bytes: int = 0) -> list:
+    """``world`` engines (ranks 0..world-1) on ``device`` in this process, peer-connected: the whole
+    multi-GPU path with merges through one device's memory. Their collective calls must be issued
+    concurrently (one host thread per engine, e.g. :func:`run_collective`)."""
+    engines = [h2tap_open(device, k, world, peer_heap_bytes) for k in range(world)]
+    try:
+        h2tap_peer_connect_local(engines)
+    except BaseException:
+        for e in engines:
+            h2tap_close(e)
+        raise
+    return engines
+
+
+def run_collective(engines, fn):
+    """Call ``fn(engine)`` for every engine concurrently (one thread each: collectives need every
+    rank's launch); returns the results in rank order, re-raising the first exception."""
+    import threading
+    out, err = [None] * len(engines), [None] * len(engines)
+
+    def work(k):
+        try:
+            out[k] = fn(engines[k])
+        except BaseException as x:  # noqa: BLE001 (re-raised below)
+            err[k] = x
+
+    ts = [threading.Thread(target=work, args=(k,)) for k in range(len(engines))]
+    for t in ts:
+        t.start()
+    for t in ts:
+        t.join()
+    for x in err:
+        if x is not None:
+            raise x
+    return out
+
+
+def connect_torch_group(engine: Engine, group=None) -> None:
+    """Multi-process bootstrap: exchange the ranks' peer handles over an initialised
+    torch.distributed process group (plumbing only), then map the segments."""
+    import torch.distributed as dist
+    handles = [None] * engine.world
+    dist.all_gather_object(handles, h2tap_peer_handle(engine), group=group)
+    h2tap_peer_connect(engine, handles)
 
 
 def h2tap_close(engine: Engine) -> None:
@@ -380,6 +445,7 @@ class Result:
         self.rows_scanned, self.device_ms, self.e2e_ms = r.rows_scanned, r.device_ms, r.e2e_ms
         self.kernel_launches = r.kernel_launches
         self.plan_flags = r.plan_flags
+        self.row_offset, self.total_rows = r.row_offset, r.total_rows
         self._columns = self._nulls = self._kernels = None
 
     def _materialise(self):

@@ -1,7 +1,7 @@
 """Build libh2tap.so in-tree with nvcc for sm_100a (B200) only.
 
-One object per csrc/*.cu (compiled in parallel), linked with the static CUDA runtime and the
-NCCL that torch ships (same libnccl.so.2 the process already has loaded under torch.distributed).
+One object per csrc/*.cu (compiled in parallel), linked with the static CUDA runtime. The cross-GPU
+merge is the library's own peer-memory kernels (csrc/peer.cuh), so nothing else is linked.
 """
 from __future__ import annotations
 
@@ -27,15 +27,6 @@ def _nvcc() -> str:
     raise RuntimeError("nvcc not found")
 
 
-def _nccl_dirs():
-    import nvidia.nccl as nn  # torch's NCCL wheel (nvidia-nccl-cu12)
-    base = list(nn.__path__)[0]
-    inc, lib = os.path.join(base, "include"), os.path.join(base, "lib")
-    if not os.path.exists(os.path.join(inc, "nccl.h")):
-        raise RuntimeError(f"nccl.h not found under {inc}")
-    return inc, lib
-
-
 def _sources():
     return sorted(glob.glob(os.path.join(CSRC, "*.cu")))
 
@@ -55,10 +46,9 @@ def build(force: bool = False, verbose: bool = False) -> str:
     if not force and not is_stale():
         return LIB
     nvcc = _nvcc()
-    nccl_inc, nccl_lib = _nccl_dirs()
     os.makedirs(BUILD, exist_ok=True)
     common = ARCH + ["-O3", "-lineinfo", "-std=c++17", "-Xcompiler", "-fPIC,-O3",
-                     "-Xptxas", "-v" if verbose else "-O3", "-I", INCLUDE, "-I", nccl_inc,
+                     "-Xptxas", "-v" if verbose else "-O3", "-I", INCLUDE,
                      "--expt-relaxed-constexpr"]
 
     def compile_one(src):
@@ -76,8 +66,7 @@ def build(force: bool = False, verbose: bool = False) -> str:
             print(err)
     objs = [o for o, _ in results]
     tmp = LIB + f".{os.getpid()}.tmp"
-    cmd = [nvcc] + ARCH + ["-shared", "-cudart", "static", "-o", tmp] + objs + [
-        "-L", nccl_lib, "-l:libnccl.so.2", "-Xlinker", f"-rpath,{nccl_lib}"]
+    cmd = [nvcc] + ARCH + ["-shared", "-cudart", "static", "-o", tmp] + objs
     r = subprocess.run(cmd, capture_output=True, text=True)
     if r.returncode != 0:
         raise RuntimeError(f"link failed:\n{r.stdout}\n{r.stderr}")

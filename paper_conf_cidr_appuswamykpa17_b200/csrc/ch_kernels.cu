@@ -17,6 +17,7 @@
 
 #include "join_index.cuh"
 #include "kernels.cuh"
+#include "peer.cuh"
 
 namespace h2tap {
 namespace {
@@ -187,16 +188,28 @@ __global__ void __launch_bounds__(kEmitThreads) sg_emit_kernel(SmallGroups g) {
 }
 
 // multi-GPU: fold another rank's (dense + sparse) tables into this rank's
-__global__ void sg_merge_kernel(const unsigned long long *__restrict__ dense,
-                                const unsigned long long *__restrict__ gtag,
-                                const unsigned long long *__restrict__ gacc, SmallGroups g) {
+// Multi-GPU (a7): every rank pushed its whole table (dense | gtag | gacc, launch_peer_push) into
+// this rank's mailbox (arrival awaited by launch_peer_wait); fold the OTHER ranks' tables into the
+// local one.
+__global__ void sg_peer_merge_kernel(PeerArgs p, SmallGroups g) {
+    pdl_wait();
+    pdl_trigger();
+    const unsigned long long seq = peer::cur_seq(p);
     const int i = blockIdx.x * blockDim.x + threadIdx.x;
-    if (i < 3 * kSgDense) {
-        if (dense[i]) atomicAdd(g.dense + i, dense[i]);
-    } else if (i < 3 * kSgDense + kSgSlots) {
-        const int s = i - 3 * kSgDense;
-        const unsigned long long t = gtag[s];
-        if (t) sg_global_add(g, (int)(unsigned int)t, gacc[3 * s], gacc[3 * s + 1], gacc[3 * s + 2]);
+    for (int k = 0; k < p.world; ++k) {
+        if (k == p.rank) continue;
+        const unsigned long long *t = reinterpret_cast<const unsigned long long *>(
+            peer::mbox(p, p.rank, (int)(seq & 1), k) + 16);
+        const unsigned long long *dense = t, *gtag = t + 3 * kSgDense, *gacc = gtag + kSgSlots;
+        if (i < 3 * kSgDense) {
+            const unsigned long long v = __ldcg(dense + i);
+            if (v) atomicAdd(g.dense + i, v);
+        } else if (i < 3 * kSgDense + kSgSlots) {
+            const int s = i - 3 * kSgDense;
+            const unsigned long long tg = __ldcg(gtag + s);
+            if (tg) sg_global_add(g, (int)(unsigned int)tg, __ldcg(gacc + 3 * s), __ldcg(gacc + 3 * s + 1),
+                                  __ldcg(gacc + 3 * s + 2));
+        }
     }
 }
 
@@ -452,9 +465,8 @@ void launch_sg_emit(const SmallGroups &g, cudaStream_t st) {
     sg_emit_kernel<<<1, kEmitThreads, 0, st>>>(g);
     count_launches(1);
 }
-void launch_sg_merge(const unsigned long long *dense, const unsigned long long *gtag,
-                     const unsigned long long *gacc, const SmallGroups &g, cudaStream_t st) {
-    sg_merge_kernel<<<(3 * kSgDense + kSgSlots + 255) / 256, 256, 0, st>>>(dense, gtag, gacc, g);
+void launch_sg_peer_merge(const PeerArgs &p, const SmallGroups &g, cudaStream_t st) {
+    launch_pdl(sg_peer_merge_kernel, (3 * kSgDense + kSgSlots + 255) / 256, 256, 0, st, p, g);
     count_launches(1);
 }
 
@@ -503,11 +515,6 @@ int q14_max_blocks(int num_sms) { return num_sms * 8; }
 void launch_q14(const int64_t *deliv, const int32_t *i_id, const int64_t *amt, uint64_t n, int64_t d_lo,
                 int64_t d_hi, const ItemMap &m, const Q14Scratch &s, int num_sms, cudaStream_t st) {
     const bool smem_map = m.words <= (uint64_t)kQ14SmemWords;
-    static bool attr = false;
-    if (!attr) {
-        cudaFuncSetAttribute(q14_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, kQ14SmemWords * 4);
-        attr = true;
-    }
     // 4 blocks per SM (each copies the map into shared memory; more blocks measured slower)
     const int per_sm = smem_map ? (m.words * 4 > (48u << 10) ? 2 : 4) : 8;
     const unsigned grid = grid_for((n + 3) / 4, kThreads, num_sms, per_sm);
@@ -526,6 +533,40 @@ void launch_q14(const int64_t *deliv, const int32_t *i_id, const int64_t *amt, u
 void launch_q14_finalize(const Q14Scratch &s, cudaStream_t st) {
     q14_finalize_kernel<<<1, 1, 0, st>>>(s.out, s.promo);
     count_launches(1);
+}
+
+// Load every kernel of this file now (CUDA lazy loading would otherwise load a kernel at its first
+// launch, which waits for the device to idle — with N logical ranks on one device, behind another
+// rank's kernel that is waiting for this rank: a deadlock).
+static cudaError_t force_load(const void *const *fs, size_t n) {
+    for (size_t i = 0; i < n; ++i) {
+        cudaFuncAttributes a;
+        const cudaError_t e = cudaFuncGetAttributes(&a, fs[i]);
+        if (e != cudaSuccess) return e;
+    }
+    return cudaSuccess;
+}
+
+cudaError_t set_attributes_ch(int num_sms) {
+    static const void *const kKernels[] = {
+        (const void *)item_map_clear_kernel,
+        (const void *)item_map_kernel,
+        (const void *)jx_build_orders_kernel,
+        (const void *)jx_clear_kernel,
+        (const void *)q12_probe_kernel,
+        (const void *)q14_finalize_kernel,
+        (const void *)q14_kernel<false>,
+        (const void *)q14_kernel<true>,
+        (const void *)q4_count_kernel,
+        (const void *)q4_mark_kernel,
+        (const void *)sg_emit_kernel,
+        (const void *)sg_peer_merge_kernel,
+        (const void *)sg_reset_kernel};
+    const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
+    if (le != cudaSuccess) return le;
+
+    (void)num_sms;
+    return cudaFuncSetAttribute(q14_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, kQ14SmemWords * 4);
 }
 
 }  // namespace h2tap

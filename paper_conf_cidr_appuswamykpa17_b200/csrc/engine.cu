@@ -1,5 +1,5 @@
 // engine.cu — the C ABI (include/h2tap.h): snapshot store in HBM with epoch publish (a1),
-// plan executors for CH Q1 / Q6 / Q18 (a2-a6, a8), NCCL merge across ranks (a7).
+// plan executors for CH Q1 / Q6 / Q18 (a2-a6, a8), the cross-GPU merge over peer segments (a7).
 //
 // Paper anchors:
 //  - snapshot = shallow copy of the top-level container + epoch++ (L562-567); here a View is
@@ -26,7 +26,6 @@
 #include <vector>
 
 #include <cuda_runtime.h>
-#include <nccl.h>
 
 #include "../../include/h2tap.h"
 #include "kernels.cuh"
@@ -75,13 +74,6 @@ struct Fail {  // thrown internally, converted to a status at the ABI boundary
         if (e_ != cudaSuccess)                                                             \
             raise(e_ == cudaErrorMemoryAllocation ? H2TAP_ENOMEM : H2TAP_ECUDA, "%s: %s (%s:%d)", \
                   #call, cudaGetErrorString(e_), __FILE__, __LINE__);                      \
-    } while (0)
-#define NK(call)                                                                           \
-    do {                                                                                   \
-        ncclResult_t r_ = (call);                                                          \
-        if (r_ != ncclSuccess)                                                             \
-            raise(H2TAP_ENCCL, "%s: %s (%s:%d)", #call, ncclGetErrorString(r_), __FILE__,  \
-                  __LINE__);                                                               \
     } while (0)
 
 // ============================================================== schema ===
@@ -310,18 +302,31 @@ struct Staging {  // pinned ring for pageable host buffers
 };
 
 // ============================================================ scratch ===
-struct Arena {  // grow-only named device buffers, owned by the engine
-    std::map<std::string, DevBufP> bufs;
+struct Arena {  // grow-only named device buffers, owned by the engine, stream-ordered on `owner`
+    struct Buf { void *ptr = nullptr; size_t bytes = 0; };
+    std::map<std::string, Buf> bufs;
     int device = 0;
+    cudaStream_t owner = nullptr;  // every use of these buffers is on this stream
     void *get(const std::string &name, size_t bytes, bool zero = false, cudaStream_t st = nullptr) {
-        auto &b = bufs[name];
-        if (!b || b->bytes < bytes) {
-            if (b) CK(cudaDeviceSynchronize());  // old buffer may still be in use on a stream
-            b.reset();
-            b = dev_alloc(bytes, device);
-            if (zero) CK(cudaMemsetAsync(b->ptr, 0, b->bytes, st));
+        Buf &b = bufs[name];
+        if (!b.ptr || b.bytes < bytes) {
+            // growth without any synchronisation: the old buffer is released after its last use
+            // in stream order and the new one comes from the stream-ordered pool. (A cudaFree or
+            // cudaDeviceSynchronize here would wait for every stream of the device — with N
+            // logical ranks on one GPU, for another rank's kernel that waits for this rank's next
+            // launch: a deadlock.)
+            if (b.ptr) CK(cudaFreeAsync(b.ptr, owner));
+            b = Buf{};
+            CK(cudaMallocAsync(&b.ptr, bytes ? bytes : 16, owner));
+            b.bytes = bytes;
+            if (zero) CK(cudaMemsetAsync(b.ptr, 0, b.bytes, st ? st : owner));
         }
-        return b->ptr;
+        return b.ptr;
+    }
+    void release() {
+        for (auto &kv : bufs)
+            if (kv.second.ptr) cudaFreeAsync(kv.second.ptr, owner);
+        bufs.clear();
     }
 };
 
@@ -371,7 +376,15 @@ struct h2tap_engine {
     // in-place updates copy only the dirty pages into the shadow (H2TAP_COW=full: always copy the
     // whole column — the A/B baseline of scripts/cow_bench.py)
     bool cow_full = false;
-    ncclComm_t comm = nullptr;
+    // a7: this rank's peer segment and the mapped segments of the others
+    struct Peer {
+        char *seg = nullptr;            // own segment (cudaMalloc: IPC-exportable)
+        size_t seg_bytes = 0;
+        std::vector<void *> opened;     // IPC mappings of other processes' segments
+        PeerArgs args{};
+        unsigned int *err_host = nullptr;  // pinned, mapped: kernels' transport error bits
+        bool connected = false, broken = false;
+    } peer;
     cudaStream_t compute = nullptr, copy = nullptr;
     cudaStream_t reaper = nullptr;  // stream-ordered frees of snapshot buffers
     FreeOrder free_order;
@@ -884,8 +897,11 @@ struct QueryCtx {
     Q18Cols out{};                          // device output columns (sorted)
     uint64_t n_max = 0;
     unsigned int *tie_dev = nullptr;
-    bool q18_sorted_on_host_sync = false;   // world > 1 path already knows nout
-    uint64_t nout_host = 0;
+    // world > 1: distributed ORDER BY
+    bool dist = false;
+    uint64_t dist_out_cap = 0;              // rows the output columns hold
+    unsigned int *recv_off = nullptr;       // this rank's bucket offsets in its heap
+    BucketSort bs{};
     long long *q6_out = nullptr;           // Q6 result {revenue, count} on the device
     // NEXT-2: Q14 / Q12 / Q4
     Q14Scratch q14{};
@@ -919,7 +935,8 @@ void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.block_part = static_cast<long long *>(e->arena.get("q6.part", sizeof(long long) * 2 * mb));
     s.done_counter = static_cast<unsigned int *>(e->arena.get("q6.counter", 64, true, e->compute));
     // world == 1: the kernel writes {revenue, count} straight into the result's device block and
-    // into the mapped pinned scalars (no copies); world > 1: allreduce, then one D2H copy
+    // into the mapped pinned scalars (no copies); world > 1: the rank's partial, then the peer
+    // allreduce writes both (a7)
     s.out = e->world > 1 ? static_cast<long long *>(e->arena.get("q6.out", 64))
                          : static_cast<long long *>(dev_block(e, q, 16));
     s.host_out = e->world > 1 ? nullptr : static_cast<long long *>(q.small_dev);
@@ -941,11 +958,14 @@ void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
             e->num_sms, e->compute);
         CK(cudaGetLastError());
     });
-    if (e->world > 1)
-        e->prof.run("q6_allreduce", [&] {
-            NK(ncclAllReduce(s.out, s.out, 2, ncclInt64, ncclSum, e->comm, e->compute));
+    if (e->world > 1) {
+        auto *dst = static_cast<long long *>(dev_block(e, q, 16));
+        e->prof.run("q6_peer_allreduce", [&] {
+            launch_peer_allreduce_i64(e->peer.args, s.out, 2, dst, static_cast<long long *>(q.small_dev),
+                                      e->compute);
         });
-    if (e->world > 1) CK(cudaMemcpyAsync(q.small.first, s.out, 16, cudaMemcpyDeviceToHost, e->compute));
+        q.q6_out = dst;
+    }
 }
 
 void finish_q6(h2tap_engine *e, QueryCtx &q) {
@@ -954,12 +974,15 @@ void finish_q6(h2tap_engine *e, QueryCtx &q) {
     const long long rev = sm[0], cnt = sm[1];
     r->nrows = 1;
     long long *blk;
-    if (r->on_device && e->world == 1) {  // the kernel wrote the result column already
+    if (r->on_device) {  // the scan (one GPU) or the allreduce wrote the result column already
         blk = q.q6_out;
         give_blocks_to_result(q);
     } else {
         blk = static_cast<long long *>(result_block(r, 16));
-        if (r->on_device) CK(cudaMemcpy(blk, sm, 16, cudaMemcpyHostToDevice));
+        if (r->on_device) {
+            CK(cudaMemcpyAsync(blk, sm, 16, cudaMemcpyHostToDevice, e->compute));
+            sync_compute(e);
+        }
         else { blk[0] = rev; blk[1] = cnt; }
         release_dev_blocks(e, q);
     }
@@ -1008,23 +1031,13 @@ void launch_q1_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
         CK(cudaGetLastError());
     });
     e->prof.run("q1_compact", [&] { launch_q1_compact(s, e->compute); });
-    if (e->world > 1) {  // a7: gather every rank's groups, fold into one table, re-compact
-        auto *cnt_dev = static_cast<unsigned long long *>(e->arena.get("q1.allcnt", 8ull * e->world));
-        e->prof.run("q1_allgather", [&] {
-            NK(ncclAllGather(s.ngroups, cnt_dev, 1, ncclUint64, e->comm, e->compute));
+    if (e->world > 1) {  // a7: every rank's group list into every rank's mailbox, folded, re-compacted
+        e->prof.run("q1_peer_push", [&] {
+            launch_peer_push(e->peer.args, s.groups, s.ngroups, 0, sizeof(Q1Group), e->num_sms, e->compute);
         });
-        std::vector<unsigned long long> cnts(e->world);
-        CK(cudaMemcpyAsync(cnts.data(), cnt_dev, 8ull * e->world, cudaMemcpyDeviceToHost, e->compute));
-        sync_compute(e);
-        const uint64_t gcap = *std::max_element(cnts.begin(), cnts.end());
-        auto *all = static_cast<Q1Group *>(e->arena.get("q1.all", sizeof(Q1Group) * std::max<uint64_t>(gcap, 1) * e->world));
-        e->prof.run("q1_allgather_groups", [&] {
-            if (gcap)
-                NK(ncclAllGather(s.groups, all, gcap * sizeof(Q1Group), ncclUint8, e->comm, e->compute));
-        });
-        e->prof.run("q1_merge", [&] {
-            for (int k = 0; k < e->world; ++k)
-                if (cnts[k]) launch_q1_merge(all + (uint64_t)k * gcap, cnts[k], s, e->compute);
+        e->prof.run("q1_peer_merge", [&] {
+            launch_peer_wait(e->peer.args, e->compute);
+            launch_q1_peer_merge(e->peer.args, s, e->num_sms, e->compute);
             launch_q1_compact(s, e->compute);
         });
     }
@@ -1099,11 +1112,44 @@ JoinIndex plan_index(h2tap_engine *e, const View &v, int table, bool force_hash,
     return j;
 }
 
-struct Q18Small { unsigned long long nout; unsigned int err, tie; Q18Stats st; };
+// {nout, err, tie} written by q18_publish (one GPU) or {n_mine, err, tie, -, row0, n_total} by the
+// distributed publish (world > 1), into mapped pinned memory
+struct Q18Small { unsigned long long nout; unsigned int err, tie; Q18Stats st; unsigned long long row0, n_total; };
 const char *const kQ18Names[8] = {"c_last", "c_id", "o_id", "o_entry_d", "o_ol_cnt", "amount_sum", "o_w_id", "o_d_id"};
 const uint32_t kQ18Types[8] = {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I32};
 const char *const kQ3Names[5] = {"ol_o_id", "ol_w_id", "ol_d_id", "revenue", "o_entry_d"};
 const uint32_t kQ3Types[5] = {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I64};
+
+struct ProfMarks : PhaseMarks {  // one profile mark per phase kernel (H2TAP_QUERY_PROFILE)
+    Prof &p;
+    cudaEvent_t a = nullptr;
+    std::string name;
+    explicit ProfMarks(Prof &pr) : p(pr) {}
+    void begin(const char *nm) override {
+        if (!p.on) return;
+        name = nm;
+        a = p.ev();
+        CK(cudaEventRecord(a, p.st));
+    }
+    void end() override {
+        if (!p.on) return;
+        cudaEvent_t b = p.ev();
+        CK(cudaEventRecord(b, p.st));
+        p.marks.push_back({name, {a, b}});
+    }
+};
+
+void q18_alloc_out(h2tap_engine *e, QueryCtx &q, uint64_t rows) {
+    Q18Cols &d = q.out;
+    d.c_last = static_cast<int32_t *>(dev_block(e, q, 4 * rows));
+    d.c_id = static_cast<int32_t *>(dev_block(e, q, 4 * rows));
+    d.o_id = static_cast<int32_t *>(dev_block(e, q, 4 * rows));
+    d.o_entry_d = static_cast<int64_t *>(dev_block(e, q, 8 * rows));
+    d.o_ol_cnt = static_cast<int32_t *>(dev_block(e, q, 4 * rows));
+    d.amount_sum = static_cast<int64_t *>(dev_block(e, q, 8 * rows));
+    d.o_w_id = static_cast<int32_t *>(dev_block(e, q, 4 * rows));
+    d.o_d_id = static_cast<int32_t *>(dev_block(e, q, 4 * rows));
+}
 
 void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     // a8: ORDER BY amount_sum DESC, o_entry_d, o_w_id, o_d_id, o_id, entirely on the device:
@@ -1138,33 +1184,9 @@ void q18_sort_and_emit(h2tap_engine *e, QueryCtx &q) {
     bs.big = static_cast<unsigned int *>(e->arena.get("q18.bbig", 4 * ((1 << kBucketMaxBits) + 1)));
     bs.ticket = static_cast<unsigned int *>(e->arena.get("q18.bticket", 64, true, e->compute));
     q.tie_dev = q.q18.tie;  // zeroed by q18_init / q3_init
+    q18_alloc_out(e, q, n_max);
     Q18Cols &d = q.out;
-    d.c_last = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    d.c_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    d.o_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    d.o_entry_d = static_cast<int64_t *>(dev_block(e, q, 8 * n_max));
-    d.o_ol_cnt = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    d.amount_sum = static_cast<int64_t *>(dev_block(e, q, 8 * n_max));
-    d.o_w_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    d.o_d_id = static_cast<int32_t *>(dev_block(e, q, 4 * n_max));
-    struct Marks : PhaseMarks {  // one profile mark per ORDER BY kernel
-        Prof &p;
-        cudaEvent_t a = nullptr;
-        std::string name;
-        explicit Marks(Prof &pr) : p(pr) {}
-        void begin(const char *nm) override {
-            if (!p.on) return;
-            name = nm;
-            a = p.ev();
-            CK(cudaEventRecord(a, p.st));
-        }
-        void end() override {
-            if (!p.on) return;
-            cudaEvent_t b = p.ev();
-            CK(cudaEventRecord(b, p.st));
-            p.marks.push_back({name, {a, b}});
-        }
-    } marks(e->prof);
+    ProfMarks marks(e->prof);
     if (e->order_v1) {
         q18_bucket_order(q.rows, q.amt, q.plan_dev, n_max, bb, bs, d, q.tie_dev, e->num_sms, e->compute,
                          &marks);
@@ -1257,90 +1279,52 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     q18_gather_and_order(e, q, n_o);
 }
 
-// a7 + a8 of Q18 (and Q3): with world > 1 gather every rank's result rows to rank 0, then the
-// ORDER BY on the device and the scalar read-backs. `n_rows_max` bounds the local row count.
+// a7 + a8 of Q18 (and Q3) with world > 1: the distributed ORDER BY. Every rank
+// ends up with its range of the global order; nothing is gathered, nothing waits for the host.
+void q18_order_dist(h2tap_engine *e, QueryCtx &q) {
+    Q18Scratch &s = q.q18;
+    const uint64_t n_max = std::max<uint64_t>(q.n_max, 1);
+    const size_t nbm = size_t(1) << kBucketMaxBits;
+    q.plan_dev = static_cast<Q18Plan *>(e->arena.get("q18.plan", sizeof(Q18Plan)));
+    BucketSort &bs = q.bs;
+    bs = BucketSort{};
+    bs.count = static_cast<unsigned int *>(e->arena.get("q18.bcount", 4 * (nbm + 1)));
+    bs.offset = static_cast<unsigned int *>(e->arena.get("q18.boffset", 4 * (nbm + 1)));
+    bs.big = static_cast<unsigned int *>(e->arena.get("q18.bbig", 4 * (nbm + 1)));
+    bs.ticket = static_cast<unsigned int *>(e->arena.get("q18.bticket", 64, true, e->compute));
+    bs.mat = static_cast<unsigned int *>(e->arena.get("q18.bmat", 4ull * ob_grid(e->num_sms) * nbm));
+    bs.kv = static_cast<unsigned long long *>(e->arena.get("q18.kv", 16 * n_max));
+    auto *send = static_cast<unsigned long long *>(e->arena.get("q18.dsend", 8 * nbm));
+    q.recv_off = static_cast<unsigned int *>(e->arena.get("q18.drecv", 4 * (nbm + 1)));
+    // output capacity: ~1/world of the global result lands here; twice the local orders rows
+    // covers any balanced sharding (more: kPeerErrOutCap, re-emitted into exact columns at finish)
+    uint64_t cap = 2 * n_max + 4096;
+    if (const char *c = std::getenv("H2TAP_DIST_OUT_CAP")) cap = std::strtoull(c, nullptr, 10);
+    q.dist_out_cap = cap;
+    q18_alloc_out(e, q, std::max<uint64_t>(cap, 1));
+    const char *cv = std::getenv("H2TAP_ORDER_CARRY");
+    const bool carry = !(cv && cv[0] == '0');
+    q.tie_dev = s.tie;
+    const Q18PlanArgs meta{s.stats, q.zone, s.nout, carry ? 1 : 0};
+    ProfMarks marks(e->prof);
+    q18_bucket_order_dist(e->peer.args, q.rows, q.amt, q.plan_dev, meta, s.err, bs, send, q.recv_off, cap, q.out,
+                          q.tie_dev, q.small_dev, e->num_sms, e->compute, &marks);
+    q.dist = true;
+}
+
+// a8 of Q18 (and Q3): the ORDER BY on the device and the scalar read-backs (mapped pinned).
+// `n_rows_max` bounds the local row count.
 void q18_gather_and_order(h2tap_engine *e, QueryCtx &q, uint64_t n_rows_max) {
     Q18Scratch &s = q.q18;
     q.rows = s.rows;
     q.amt = s.amt;
     q.n_max = n_rows_max;
-    Q18Small *sm = static_cast<Q18Small *>(q.small.first);
     if (e->world > 1) {
-        // a7: groups are warehouse-local; gather the result rows to rank 0 (host-sized NCCL calls)
-        CK(cudaMemcpyAsync(&sm->nout, s.nout, 8, cudaMemcpyDeviceToHost, e->compute));
-        CK(cudaMemcpyAsync(&sm->err, s.err, 4, cudaMemcpyDeviceToHost, e->compute));
-        sync_compute(e);
-        int err_any = sm->err ? 1 : 0;
-        auto *flag = static_cast<int *>(e->arena.get("q18.errflag", 64));
-        CK(cudaMemcpyAsync(flag, &err_any, 4, cudaMemcpyHostToDevice, e->compute));
-        NK(ncclAllReduce(flag, flag, 1, ncclInt32, ncclMax, e->comm, e->compute));
-        CK(cudaMemcpyAsync(&err_any, flag, 4, cudaMemcpyDeviceToHost, e->compute));
-        sync_compute(e);
-        if (sm->err) return;  // finish raises the local error
-        if (err_any) raise(H2TAP_EPLAN, "Q%u: failed on another rank", q.plan);
-        {   // the ORDER BY bounds must cover every rank's rows: min/max of the zones
-            static_assert(sizeof(Q18Zone) == 12 * sizeof(int), "Q18Zone: 6 (min, max) int pairs");
-            int zmin[6], zmax[6];
-            const int *zp = reinterpret_cast<const int *>(&q.zone);
-            for (int k = 0; k < 6; ++k) { zmin[k] = zp[2 * k]; zmax[k] = zp[2 * k + 1]; }
-            auto *zd = static_cast<int *>(e->arena.get("q18.zone", 64));
-            CK(cudaMemcpyAsync(zd, zmin, 24, cudaMemcpyHostToDevice, e->compute));
-            CK(cudaMemcpyAsync(zd + 6, zmax, 24, cudaMemcpyHostToDevice, e->compute));
-            NK(ncclAllReduce(zd, zd, 6, ncclInt32, ncclMin, e->comm, e->compute));
-            NK(ncclAllReduce(zd + 6, zd + 6, 6, ncclInt32, ncclMax, e->comm, e->compute));
-            CK(cudaMemcpyAsync(zmin, zd, 24, cudaMemcpyDeviceToHost, e->compute));
-            CK(cudaMemcpyAsync(zmax, zd + 6, 24, cudaMemcpyDeviceToHost, e->compute));
-            sync_compute(e);
-            int *zw = reinterpret_cast<int *>(&q.zone);
-            for (int k = 0; k < 6; ++k) { zw[2 * k] = zmin[k]; zw[2 * k + 1] = zmax[k]; }
-        }
-        auto *cnt_dev = static_cast<unsigned long long *>(e->arena.get("q18.allcnt", 8ull * e->world));
-        NK(ncclAllGather(s.nout, cnt_dev, 1, ncclUint64, e->comm, e->compute));
-        std::vector<unsigned long long> cnts(e->world);
-        CK(cudaMemcpyAsync(cnts.data(), cnt_dev, 8ull * e->world, cudaMemcpyDeviceToHost, e->compute));
-        sync_compute(e);
-        uint64_t total = 0;
-        for (auto c : cnts) total += c;
-        Q18Row *all = e->rank == 0 ? static_cast<Q18Row *>(e->arena.get("q18.allrows", sizeof(Q18Row) * std::max<uint64_t>(total, 1)))
-                                   : nullptr;
-        long long *all_amt = e->rank == 0 ? static_cast<long long *>(e->arena.get("q18.allamt", 8 * std::max<uint64_t>(total, 1)))
-                                          : nullptr;
-        e->prof.run("q18_gather", [&] {
-            NK(ncclGroupStart());
-            uint64_t off = 0;
-            for (int k = 0; k < e->world; ++k) {
-                const size_t bytes = cnts[k] * sizeof(Q18Row), abytes = cnts[k] * 8;
-                if (bytes) {
-                    if (e->rank == 0 && k == 0) {
-                        CK(cudaMemcpyAsync(all, s.rows, bytes, cudaMemcpyDeviceToDevice, e->compute));
-                        CK(cudaMemcpyAsync(all_amt, s.amt, abytes, cudaMemcpyDeviceToDevice, e->compute));
-                    } else if (e->rank == 0) {
-                        NK(ncclRecv(all + off, bytes, ncclUint8, k, e->comm, e->compute));
-                        NK(ncclRecv(all_amt + off, abytes, ncclUint8, k, e->comm, e->compute));
-                    } else if (e->rank == k) {
-                        NK(ncclSend(s.rows, bytes, ncclUint8, 0, e->comm, e->compute));
-                        NK(ncclSend(s.amt, abytes, ncclUint8, 0, e->comm, e->compute));
-                    }
-                }
-                off += cnts[k];
-            }
-            NK(ncclGroupEnd());
-        });
-        if (e->rank != 0) {  // rows are returned on rank 0 only
-            q.q18_sorted_on_host_sync = true;
-            q.nout_host = 0;
-            return;
-        }
-        q.rows = all;
-        q.amt = all_amt;
-        q.n_max = total;
-        sm->nout = total;
-        CK(cudaMemcpyAsync(s.nout, &sm->nout, 8, cudaMemcpyHostToDevice, e->compute));
-        launch_q18_stats(all, all_amt, total, s, e->num_sms, e->compute);  // stats of gathered rows
+        q18_order_dist(e, q);
+        return;
     }
     q18_sort_and_emit(e, q);
-    launch_q18_publish(s.nout, s.err, q.tie_dev, q.small_dev, e->compute);  // -> sm (mapped)
-    (void)sm;
+    launch_q18_publish(s.nout, s.err, q.tie_dev, q.small_dev, e->compute);  // -> small (mapped)
 }
 
 // ---- NEXT-2: CH Q3 (customer ⋈ new_order ⋈ orders ⋈ order_line) on the Q18 machinery
@@ -1398,19 +1382,36 @@ void finish_q18(h2tap_engine *e, QueryCtx &q) {
     const char *const *names = q3 ? kQ3Names : kQ18Names;
     const uint32_t *types = q3 ? kQ3Types : kQ18Types;
     const int ncols = q3 ? 5 : 8;
-    if (q.q18_sorted_on_host_sync) {  // world > 1, rank != 0
-        r->nrows = 0;
-        for (int i = 0; i < ncols; ++i) add_col(r, names[i], types[i], result_block(r, 8));
-        release_dev_blocks(e, q);
-        return;
-    }
-    const unsigned int err = sm->err;
+    const unsigned int err = sm->err;  // world > 1: every rank's join errors and the exchange's
     const unsigned pl = q.plan;
+    if (err & kPeerErrTimeout) {
+        e->peer.broken = true;
+        raise(H2TAP_EPEER, "Q%u: a peer did not deliver its ORDER BY exchange in time", pl);
+    }
     if (err & kErrDupOrders) raise(H2TAP_EDUPKEY, "Q%u: duplicate orders primary key (w, d, o_id)", pl);
     if (err & kErrDupCustomer) raise(H2TAP_EDUPKEY, "Q%u: duplicate customer primary key (w, d, c_id)", pl);
     if (err & kErrDomain) raise(H2TAP_EPLAN, "Q%u: join key outside the supported domain", pl);
+    if (err & kPeerErrHeap)
+        raise(H2TAP_ENOMEM, "Q%u: a rank's share of the distributed ORDER BY exceeds its peer heap "
+              "(h2tap_config.peer_heap_bytes)", pl);
+    if (err & kPeerErrNoCarry)
+        raise(H2TAP_EPLAN, "Q%u: the distributed ORDER BY needs 128-bit carry records; the result "
+              "fields are too wide", pl);
     const uint64_t nout = sm->nout;
-    if (sm->tie && nout > 1) {
+    r->total_rows = q.dist ? sm->n_total : nout;
+    r->row_offset = q.dist ? sm->row0 : 0;
+    if (q.dist && (err & kPeerErrOutCap)) {
+        // this rank's slice exceeded the output columns: re-emit from the heap into exact ones
+        // (the exchanged records stay there until the next exchange of the same parity)
+        release_dev_blocks(e, q);
+        q18_alloc_out(e, q, std::max<uint64_t>(nout, 1));
+        const unsigned int cleared = err & ~kPeerErrOutCap;
+        CK(cudaMemcpyAsync(reinterpret_cast<char *>(q.plan_dev) + offsetof(Q18Plan, err), &cleared, 4,
+                           cudaMemcpyHostToDevice, e->compute));
+        q18_dist_emit(e->peer.args, q.plan_dev, q.recv_off, q.out, q.tie_dev, q.bs, e->num_sms, e->compute);
+        sync_compute(e);
+    }
+    if (!q.dist && sm->tie && nout > 1) {
         // a run of > 32 equal 64-bit prefixes, or a bucket larger than shared memory: redo
         // exactly, one stable LSD radix sort per field (r, then e, then a)
         SortPairs w = q.sp;
@@ -1498,8 +1499,8 @@ void launch_q14_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
         CK(cudaGetLastError());
     });
     if (e->world > 1)
-        e->prof.run("q14_allreduce", [&] {
-            NK(ncclAllReduce(s.out, s.out, 3, ncclInt64, ncclSum, e->comm, e->compute));
+        e->prof.run("q14_peer_allreduce", [&] {
+            launch_peer_allreduce_i64(e->peer.args, s.out, 3, s.out, nullptr, e->compute);
         });
     e->prof.run("q14_finalize", [&] { launch_q14_finalize(s, e->compute); });
     auto *sm = static_cast<Q14Small *>(q.small.first);
@@ -1516,7 +1517,8 @@ void finish_q14(h2tap_engine *e, QueryCtx &q) {
     const bool null = sm->out[2] == 0;  // SUM over no joined row IS NULL -> NULL ratio (R30)
     auto *blk = static_cast<long long *>(result_block(r, 32));
     if (r->on_device) {
-        CK(cudaMemcpy(blk, sm->out, 24, cudaMemcpyHostToDevice));
+        CK(cudaMemcpyAsync(blk, sm->out, 24, cudaMemcpyHostToDevice, e->compute));
+        sync_compute(e);
         add_col(r, "promo_revenue", H2TAP_F64, q.q14.promo);
         give_blocks_to_result(q);
     } else {
@@ -1554,17 +1556,13 @@ void sg_setup(h2tap_engine *e, QueryCtx &q) {
 
 void sg_merge_and_emit(h2tap_engine *e, QueryCtx &q, const char *name) {
     SmallGroups &g = q.sg;
-    if (e->world > 1) {  // a7: every rank's tables to every rank, folded into the local one
+    if (e->world > 1) {  // a7: every rank's tables to every rank's mailbox, folded into the local one
         const size_t words = 3 * kSgDense + 4 * kSgSlots;
-        auto *all = static_cast<unsigned long long *>(e->arena.get("sg.all", 8ull * words * e->world));
-        e->prof.run((std::string(name) + "_allgather").c_str(), [&] {
-            NK(ncclAllGather(g.dense, all, words, ncclUint64, e->comm, e->compute));
+        e->prof.run((std::string(name) + "_peer_merge").c_str(), [&] {
+            launch_peer_push(e->peer.args, g.dense, nullptr, words, 8u, e->num_sms, e->compute);
+            launch_peer_wait(e->peer.args, e->compute);
+            launch_sg_peer_merge(e->peer.args, g, e->compute);
         });
-        for (int k = 0; k < e->world; ++k)
-            if (k != e->rank) {
-                const unsigned long long *t = all + (size_t)k * words;
-                launch_sg_merge(t, t + 3 * kSgDense, t + 3 * kSgDense + kSgSlots, g, e->compute);
-            }
     }
     e->prof.run((std::string(name) + "_emit").c_str(), [&] { launch_sg_emit(g, e->compute); });
     auto *sm = static_cast<SgSmall *>(q.small.first);
@@ -1718,6 +1716,9 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
     }
     std::lock_guard<std::mutex> g(e->query_mu);
     CK(cudaSetDevice(e->device));
+    if (e->world > 1 && (!e->peer.connected || e->peer.broken))
+        return fail(H2TAP_EPEER, e->peer.broken ? "the peer group failed earlier (close and re-open the engines)"
+                                                : "world > 1: call h2tap_peer_connect / h2tap_peer_connect_local first");
     publish_ready(e, false);
     ViewP v;
     {
@@ -1766,6 +1767,12 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
     auto finish_upto = [&](size_t upto) {
         if (done >= upto) return;
         sync_compute(e);
+        if (e->world > 1 && *reinterpret_cast<volatile unsigned int *>(e->peer.err_host)) {
+            e->peer.broken = true;
+            const volatile unsigned int *d = e->peer.err_host;
+            raise(H2TAP_EPEER, "rank %d: rank %u did not deliver cross-GPU merge #%u within %.0f ms (its "
+                  "flag here: %u)", e->rank, d[2], d[1], e->peer.args.timeout_ns / 1e6, d[3]);
+        }
         for (; done < upto; ++done) {
             QueryCtx &q = ctx[done];
             switch (q.plan) {
@@ -1821,6 +1828,7 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
             r->kms.push_back(k);
         }
         r->e2e_ms = wall;
+        if (!q.dist) r->total_rows = r->nrows;
         e->host_pool->put(q.small.first, q.small.second);
         q.small = {};
     }
@@ -1861,8 +1869,8 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         *out = nullptr;
         if (cfg->world < 1 || cfg->rank < 0 || cfg->rank >= cfg->world)
             return fail(H2TAP_EINVAL, "bad rank %d / world %d", cfg->rank, cfg->world);
-        if (cfg->world > 1 && !cfg->nccl_unique_id)
-            return fail(H2TAP_EINVAL, "world > 1 needs an NCCL unique id");
+        if (cfg->world > kMaxRanks)
+            return fail(H2TAP_EINVAL, "world %d > %d ranks (one node)", cfg->world, kMaxRanks);
         int ndev = 0;
         CK(cudaGetDeviceCount(&ndev));
         if (cfg->device < 0 || cfg->device >= ndev)
@@ -1878,6 +1886,13 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
             return fail(H2TAP_ECUDA, "built for sm_100a (B200); device %d is sm_%d%d", e->device,
                         prop.major, prop.minor);
         e->num_sms = prop.multiProcessorCount;
+        CK(set_attributes_scan(e->num_sms));  // per device: shared-memory limits of the kernels
+        CK(set_attributes_join(e->num_sms));
+        CK(set_attributes_sort(e->num_sms));
+        CK(set_attributes_ch(e->num_sms));
+        CK(set_attributes_layout(e->num_sms));
+        CK(set_attributes_store(e->num_sms));
+        CK(set_attributes_peer(e->num_sms));
         if (const char *impl = std::getenv("H2TAP_SCAN")) e->scan_tma = std::strcmp(impl, "ldg") != 0;
         if (const char *ob = std::getenv("H2TAP_ORDER")) e->order_v1 = std::strcmp(ob, "v1") == 0;
         if (const char *z = std::getenv("H2TAP_ZC_TMA")) e->zc_tma = std::atoi(z) != 0;
@@ -1906,12 +1921,31 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         CK(cudaMallocHost(&e->small_host, 256));
         e->arena.device = e->device;
         e->load_arena.device = e->device;
+        e->arena.owner = e->compute;
+        e->load_arena.owner = e->copy;
         e->host_pool = std::make_shared<BlockPool>(true, e->device);
         e->dev_pool = std::make_shared<BlockPool>(false, e->device);
-        if (e->world > 1) {
-            ncclUniqueId id;
-            std::memcpy(&id, cfg->nccl_unique_id, sizeof id);
-            NK(ncclCommInitRank(&e->comm, e->world, id, e->rank));
+        if (e->world > 1) {  // a7: this rank's peer segment, zeroed before any peer maps it
+            auto &P = e->peer;
+            uint64_t heap = cfg->peer_heap_bytes ? cfg->peer_heap_bytes : (1ull << 30);
+            const uint64_t half = ((heap / 2) + 255) & ~uint64_t(255);
+            P.seg_bytes = kPeerCtlBytes + 2 * kMaxRanks * kPeerSlotBytes + 2 * half;
+            CK(cudaMalloc(&P.seg, P.seg_bytes));
+            CK(cudaMemset(P.seg, 0, kPeerCtlBytes));
+            CK(cudaHostAlloc(&P.err_host, 64, cudaHostAllocMapped));
+            *P.err_host = 0;
+            CK(cudaDeviceSynchronize());
+            P.args = PeerArgs{};
+            P.args.rank = e->rank;
+            P.args.world = e->world;
+            P.args.slot_bytes = kPeerSlotBytes;
+            P.args.heap_half = half;
+            double ms = 20000.0;
+            if (const char *t = std::getenv("H2TAP_PEER_TIMEOUT_MS")) ms = std::atof(t);
+            P.args.timeout_ns = (unsigned long long)(ms * 1e6);
+            void *dp = nullptr;
+            CK(cudaHostGetDevicePointer(&dp, P.err_host, 0));
+            P.args.err_host = static_cast<unsigned int *>(dp);
         }
         *out = e.release();
         return H2TAP_OK;
@@ -2151,7 +2185,9 @@ void h2tap_close(h2tap_engine *e) {
     try { publish_ready(e, true); } catch (...) {}
     cudaStreamSynchronize(e->compute);
     cudaStreamSynchronize(e->copy);
-    if (e->comm) ncclCommDestroy(e->comm);
+    for (void *p : e->peer.opened) cudaIpcCloseMemHandle(p);
+    if (e->peer.seg) cudaFree(e->peer.seg);
+    if (e->peer.err_host) cudaFreeHost(e->peer.err_host);
     for (auto &p : e->pending) {
         for (cudaEvent_t ev : {p.done, p.t0, p.t1, p.t2, p.t3}) cudaEventDestroy(ev);
         e->host_pool->put(p.stats_block.first, p.stats_block.second);
@@ -2167,8 +2203,10 @@ void h2tap_close(h2tap_engine *e) {
     e->published.reset();
     e->accepted.reset();
     for (auto &t : e->tables) for (auto &c : t.col) { c.cur.reset(); c.alt.reset(); c.bits.reset(); c.bits_next.reset(); }
-    e->arena.bufs.clear();
-    e->load_arena.bufs.clear();
+    e->arena.release();
+    e->load_arena.release();
+    cudaStreamSynchronize(e->compute);
+    cudaStreamSynchronize(e->copy);
     cudaStreamSynchronize(e->reaper);
     cudaStreamDestroy(e->compute);
     cudaStreamDestroy(e->copy);
@@ -2178,13 +2216,68 @@ void h2tap_close(h2tap_engine *e) {
 
 const char *h2tap_last_error(void) { return g_err.c_str(); }
 
-h2tap_status h2tap_nccl_unique_id(void *out128) {
-    if (!out128) return fail(H2TAP_EINVAL, "out is NULL");
+h2tap_status h2tap_peer_handle(h2tap_engine *e, void *out64) {
     return guarded([&]() -> h2tap_status {
-        ncclUniqueId id;
-        NK(ncclGetUniqueId(&id));
-        static_assert(sizeof(ncclUniqueId) == 128, "ncclUniqueId is 128 bytes");
-        std::memcpy(out128, &id, sizeof id);
+        if (!e || !out64) return fail(H2TAP_EINVAL, "engine/out is NULL");
+        if (e->world < 2) return fail(H2TAP_EINVAL, "world == 1: no peer segment");
+        CK(cudaSetDevice(e->device));
+        cudaIpcMemHandle_t h;
+        static_assert(sizeof(cudaIpcMemHandle_t) == 64, "CUDA IPC handles are 64 bytes");
+        CK(cudaIpcGetMemHandle(&h, e->peer.seg));
+        std::memcpy(out64, &h, 64);
+        return H2TAP_OK;
+    });
+}
+
+h2tap_status h2tap_peer_connect(h2tap_engine *e, const void *handles, uint32_t world) {
+    return guarded([&]() -> h2tap_status {
+        if (!e || !handles) return fail(H2TAP_EINVAL, "engine/handles is NULL");
+        if ((int)world != e->world || e->world < 2) return fail(H2TAP_EINVAL, "world %u != engine world %d", world, e->world);
+        if (e->peer.connected) return fail(H2TAP_EINVAL, "peers already connected");
+        CK(cudaSetDevice(e->device));
+        auto &P = e->peer;
+        for (int k = 0; k < e->world; ++k) {
+            if (k == e->rank) { P.args.seg[k] = P.seg; continue; }
+            cudaIpcMemHandle_t h;
+            std::memcpy(&h, static_cast<const char *>(handles) + 64 * k, 64);
+            void *p = nullptr;
+            CK(cudaIpcOpenMemHandle(&p, h, cudaIpcMemLazyEnablePeerAccess));
+            P.opened.push_back(p);
+            P.args.seg[k] = static_cast<char *>(p);
+        }
+        P.connected = true;
+        return H2TAP_OK;
+    });
+}
+
+h2tap_status h2tap_peer_connect_local(h2tap_engine *const *engines, uint32_t n) {
+    return guarded([&]() -> h2tap_status {
+        if (!engines || n < 2 || n > (uint32_t)kMaxRanks) return fail(H2TAP_EINVAL, "need 2..%d engines", kMaxRanks);
+        for (uint32_t i = 0; i < n; ++i) {
+            if (!engines[i]) return fail(H2TAP_EINVAL, "engine %u is NULL", i);
+            if (engines[i]->rank != (int)i || engines[i]->world != (int)n)
+                return fail(H2TAP_EINVAL, "engine %u has rank %d / world %d (want %u / %u)", i, engines[i]->rank,
+                            engines[i]->world, i, n);
+            if (engines[i]->peer.connected) return fail(H2TAP_EINVAL, "engine %u already connected", i);
+        }
+        for (uint32_t i = 0; i < n; ++i) {
+            h2tap_engine *e = engines[i];
+            CK(cudaSetDevice(e->device));
+            for (uint32_t k = 0; k < n; ++k) {
+                if (engines[k]->device != e->device) {  // another GPU of this process: peer access
+                    const cudaError_t r = cudaDeviceEnablePeerAccess(engines[k]->device, 0);
+                    if (r == cudaErrorPeerAccessAlreadyEnabled) cudaGetLastError();
+                    else CK(r);
+                }
+                e->peer.args.seg[k] = engines[k]->peer.seg;
+            }
+        }
+        for (uint32_t i = 0; i < n; ++i) {
+            int shared = 0;
+            for (uint32_t k = 0; k < n; ++k) shared |= (k != i && engines[k]->device == engines[i]->device);
+            engines[i]->peer.args.shared_device = shared;
+            engines[i]->peer.connected = true;
+        }
         return H2TAP_OK;
     });
 }

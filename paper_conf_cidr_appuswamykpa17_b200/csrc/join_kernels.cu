@@ -382,17 +382,6 @@ q18_having_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o
     stat.flush(s.stat_part, s.ticket, s.stats);
 }
 
-__global__ void q18_stats_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ amt,
-                                 uint64_t n, Q18Stats *st, Q18Stats *part, unsigned int *ticket) {
-    StatAcc stat;
-    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
-        const Q18Row r = rows[i];
-        stat.add(amt[i], r);
-    }
-    stat.flush(part, ticket, st);
-}
-
 // ------------------------------------------------------------- CH Q3 (NEXT-2) --
 // Q3 = customer ⋈ new_order ⋈ orders ⋈ order_line, GROUP BY the orders key, ORDER BY revenue
 // DESC, o_entry_d. Its group key (ol_o_id, ol_w_id, ol_d_id, o_entry_d) is functionally
@@ -566,12 +555,6 @@ void launch_q3_emit(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id,
 void launch_q18_probe_tma(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
                           const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
                           cudaStream_t st) {
-    static bool init = false;
-    if (!init) {
-        cudaFuncSetAttribute(q18_probe_tma_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                             (int)sizeof(ProbeStages));
-        init = true;
-    }
     const uint64_t nchunks = (n_ol + kProbeChunk - 1) / kProbeChunk;
     const unsigned grid = (unsigned)(nchunks < (uint64_t)num_sms ? (nchunks ? nchunks : 1) : num_sms);
     q18_probe_tma_kernel<<<grid, (kProbeTmaWarps + 1) * 32, sizeof(ProbeStages), st>>>(ol_w, ol_d, ol_o,
@@ -598,11 +581,37 @@ void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_
     count_launches(1);
 }
 
-void launch_q18_stats(const Q18Row *rows, const long long *amt, uint64_t n, const Q18Scratch &s,
-                      int num_sms, cudaStream_t st) {
-    q18_stats_kernel<<<grid_for(n, 256, num_sms, 4), 256, 0, st>>>(rows, amt, n, s.stats, s.stat_part,
-                                                                  s.ticket);
-    count_launches(1);
+
+// Load every kernel of this file now (CUDA lazy loading would otherwise load a kernel at its first
+// launch, which waits for the device to idle — with N logical ranks on one device, behind another
+// rank's kernel that is waiting for this rank: a deadlock).
+static cudaError_t force_load(const void *const *fs, size_t n) {
+    for (size_t i = 0; i < n; ++i) {
+        cudaFuncAttributes a;
+        const cudaError_t e = cudaFuncGetAttributes(&a, fs[i]);
+        if (e != cudaSuccess) return e;
+    }
+    return cudaSuccess;
+}
+
+cudaError_t set_attributes_join(int num_sms) {
+    static const void *const kKernels[] = {
+        (const void *)q18_build_kernel,
+        (const void *)q18_having_kernel<2>,
+        (const void *)q18_having_kernel<4>,
+        (const void *)q18_init_kernel,
+        (const void *)q18_probe_kernel<false>,
+        (const void *)q18_probe_kernel<true>,
+        (const void *)q18_probe_tma_kernel,
+        (const void *)q18_publish_kernel,
+        (const void *)q3_emit_kernel,
+        (const void *)q3_mark_kernel};
+    const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
+    if (le != cudaSuccess) return le;
+
+    (void)num_sms;
+    return cudaFuncSetAttribute(q18_probe_tma_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                (int)sizeof(ProbeStages));
 }
 
 }  // namespace h2tap

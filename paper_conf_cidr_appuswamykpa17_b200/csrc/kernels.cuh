@@ -60,9 +60,50 @@ void launch_q61_tma(const int32_t *number, const int64_t *deliv, const int32_t *
                     int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s6, int num_sms,
                     cudaStream_t st);
 void launch_q1_compact(const Q1Scratch &s, cudaStream_t st);        // tables -> groups[], ngroups
-void launch_q1_merge(const Q1Group *all, uint64_t n, const Q1Scratch &s, cudaStream_t st);
 void launch_q1_emit(const Q1Scratch &s, uint64_t max_groups, cudaStream_t st);  // rank by key + AVG;
                                                                            // reads *ngroups on device
+
+// ----------------------------------------------------- a7 peer transport (peer.cuh) --
+// Cross-GPU merges move data with stores into the other ranks' "peer segments".
+constexpr int kMaxRanks = 8;                               // one 8-GPU node
+constexpr size_t kPeerCtlBytes = 64u << 10;
+constexpr size_t kPeerSlotBytes = (2u << 20) + (64u << 10); // >= 16 + Q1's max group list (2 MB)
+// (high bits: they share Q18Plan::err with the join error bits kErr*)
+enum : unsigned int { kPeerErrTimeout = 1u << 16, kPeerErrHeap = 1u << 17, kPeerErrNoCarry = 1u << 18,
+                      kPeerErrOutCap = 1u << 19 };
+struct PeerCtl {                     // at offset 0 of every segment
+    unsigned long long flag[kMaxRanks];  // flag[k]: last collective rank k delivered here
+    unsigned long long seq;              // last collective this rank issued (device counter)
+    unsigned int err;                    // sticky transport error bits
+    unsigned int ticket;                 // last-block counter of multi-block producers
+};
+struct PeerArgs {                    // passed by value to every merge kernel
+    char *seg[kMaxRanks];            // rank k's segment as mapped here (seg[rank] = own)
+    int rank, world;
+    unsigned long long slot_bytes, heap_half, timeout_ns;
+    unsigned int *err_host;          // mapped pinned host word: error bits visible to the host
+    // 1: another rank runs on this device in this process (N logical ranks on one GPU). A kernel
+    // that waits for peers then lets its successor launch (PDL) only after the wait: a successor
+    // resident early holds a share of every SM, which another rank's producer (one 224 KB block
+    // per SM) may need — the producer this rank is waiting for. 0: the successor
+    // launches early, as everywhere else on the hot path.
+    int shared_device;
+};
+// Sum-allreduce of n <= 8 int64 values: dst (device, may equal src) and host_dst (mapped, or null)
+void launch_peer_allreduce_i64(const PeerArgs &p, const long long *src, int n, long long *dst,
+                               long long *host_dst, cudaStream_t st);
+// Producer: copy `count` elements of `elem_bytes` (count read from *count_dev when non-null, else
+// count_const) into mailbox[s & 1][rank] of every rank, slot header = the count (u64), data at +16.
+void launch_peer_push(const PeerArgs &p, const void *src, const unsigned long long *count_dev,
+                      unsigned long long count_const, unsigned int elem_bytes, int num_sms, cudaStream_t st);
+// Consumer-only kernel (one thread): wait for every rank's latest collective; the multi-block
+// consumers that read the mailboxes / heap run after it in stream order
+void launch_peer_wait(const PeerArgs &p, cudaStream_t st);
+// Q1: fold every rank's compacted group list (mailbox) into the clean global table. Like every
+// multi-block consumer it does not wait itself: launch_peer_wait (one thread) runs before it, so
+// waiting never occupies more than one block (N logical ranks on one device: a waiting grid
+// could hold the SMs another rank's producer needs)
+void launch_q1_peer_merge(const PeerArgs &p, const Q1Scratch &s, int num_sms, cudaStream_t st);
 
 // ------------------------------------------------------------ Q18 (K3-K5) --
 struct HtSlot { unsigned long long key; unsigned int row; unsigned int pad; };  // 16 B
@@ -147,8 +188,6 @@ void launch_q3_emit(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id,
 // {nout, err, tie} -> mapped pinned host memory (one launch instead of three D2H copies)
 void launch_q18_publish(const unsigned long long *nout, const unsigned int *err, const unsigned int *tie,
                         void *host_small, cudaStream_t st);
-void launch_q18_stats(const Q18Row *rows, const long long *amt, uint64_t n, const Q18Scratch &s,
-                      int num_sms, cudaStream_t st);  // recompute stats over gathered rows (multi-GPU)
 
 // ------------------------------------------------------------------ sort ---
 // Stable LSD radix sort of (u64 key, u32 value) pairs, 8-bit digits, `bits` low key bits.
@@ -207,10 +246,20 @@ struct Q18SortSpec {         // host-computed from Q18Stats
 // (no host round trip): field widths, 64-bit prefix width, whether a tie-fix is needed, and the
 // bucket shift for `bucket_bits` buckets.
 struct Q18Plan {
-    unsigned long long n;
+    unsigned long long n;        // rows this rank sorts (world > 1: its rows BEFORE the exchange)
     Q18SortSpec spec;
     int tiefix;
     int shift;
+    int bucket_bits;             // buckets = 1 << bucket_bits (world > 1: from the global row count)
+    // distributed ORDER BY (world > 1): the buckets are range-partitioned over
+    // the ranks by their global row positions; rank k holds rows [row0, row0 + n_mine) of the
+    // globally ordered result
+    int dist;
+    unsigned int b_lo, nb_mine;  // this rank's buckets [b_lo, b_lo + nb_mine)
+    unsigned long long n_total, n_mine, row0;
+    unsigned long long xseq;     // sequence number of the record exchange (heap parity = xseq & 1)
+    unsigned long long nbuckets; // dist: 1 << bucket_bits (the length of the pushed count list)
+    unsigned int err;            // OR of every rank's join error bits (+ kErrPeer*)
 };
 void launch_q18_plan(const Q18Stats *stats, const Q18Zone &zone, const unsigned long long *nout,
                      int bucket_bits, bool allow_carry, Q18Plan *plan, unsigned int *flag,
@@ -236,6 +285,19 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, Q18Plan *plan
                          int bucket_bits, const BucketSort &s, const Q18Cols &dst, unsigned int *flag,
                          int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr,
                          const Q18PlanArgs *plan_args = nullptr);  // non-null: hist writes *plan
+// Distributed ORDER BY (world > 1): plan from every rank's statistics, local
+// partition, exchange of the carry records into the owners' heaps, per-bucket sort + emit of this
+// rank's range of the global order into dst (capacity out_cap rows); {n_mine, err, tie, stats,
+// row0, n_total} -> host_small (mapped). send: [2^kBucketMaxBits] u64, recv_off: [2^kBucketMaxBits+1].
+void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long long *amt, Q18Plan *plan,
+                           const Q18PlanArgs &meta, const unsigned int *err, const BucketSort &s,
+                           unsigned long long *send, unsigned int *recv_off, uint64_t out_cap,
+                           const Q18Cols &dst, unsigned int *flag, void *host_small, int num_sms,
+                           cudaStream_t st, PhaseMarks *marks = nullptr);
+// The emit phase alone (re-run by the host into larger output columns after kPeerErrOutCap; the
+// exchanged records stay in the heap until the next exchange of the same parity).
+void q18_dist_emit(const PeerArgs &pa, const Q18Plan *plan, const unsigned int *recv_off, const Q18Cols &dst,
+                   unsigned int *flag, const BucketSort &s, int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr);
 // Within runs of equal prefix, order by the full tuple; runs longer than 32 raise *flag.
 // Exact fallback: three stable passes over the full fields (row rank, entry, amount).
 void launch_q18_field_keys(const Q18Row *rows, const long long *amt, const unsigned int *vals,
@@ -264,6 +326,15 @@ void launch_apply_updates(void *col, uint32_t es, uint32_t *bits, const uint32_t
                           const void *vals, uint64_t n, int num_sms, cudaStream_t st);
 
 // ---------------------------------------------------------------- helpers --
+// Per file: load every kernel and set the dynamic shared-memory limits, for the current device, at
+// h2tap_open (per device, return codes checked; no per-process static flags).
+cudaError_t set_attributes_scan(int num_sms);
+cudaError_t set_attributes_join(int num_sms);
+cudaError_t set_attributes_sort(int num_sms);
+cudaError_t set_attributes_ch(int num_sms);
+cudaError_t set_attributes_layout(int num_sms);
+cudaError_t set_attributes_store(int num_sms);
+cudaError_t set_attributes_peer(int num_sms);
 // Every launcher counts the kernels it launches (reported per query as kernel_launches).
 void count_launches(int n);
 
@@ -305,8 +376,9 @@ struct SmallGroups {
 };
 void launch_sg_reset(const SmallGroups &g, cudaStream_t st);  // once, at allocation
 void launch_sg_emit(const SmallGroups &g, cudaStream_t st);   // rank + write; re-clears the tables
-void launch_sg_merge(const unsigned long long *dense, const unsigned long long *gtag,
-                     const unsigned long long *gacc, const SmallGroups &g, cudaStream_t st);
+// multi-GPU: wait for every rank's pushed table (dense | gtag | gacc contiguous, launch_peer_push)
+// and fold the other ranks' tables into g
+void launch_sg_peer_merge(const PeerArgs &p, const SmallGroups &g, cudaStream_t st);
 // orders (w, d, o_id) join index alone: clear + insert (and zero mark[] for Q4 when non-null)
 void launch_jx_build_orders(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
                             const JoinIndex &jo, unsigned int *err, uint8_t *mark, int num_sms,

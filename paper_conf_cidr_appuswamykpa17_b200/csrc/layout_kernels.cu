@@ -191,4 +191,27 @@ void launch_layout_sum(const int32_t *data, int layout, uint64_t n, int log_ncol
     count_launches(1);
 }
 
+// Load every kernel of this file now (CUDA lazy loading would otherwise load a kernel at its first
+// launch, which waits for the device to idle — with N logical ranks on one device, behind another
+// rank's kernel that is waiting for this rank: a deadlock).
+static cudaError_t force_load(const void *const *fs, size_t n) {
+    for (size_t i = 0; i < n; ++i) {
+        cudaFuncAttributes a;
+        const cudaError_t e = cudaFuncGetAttributes(&a, fs[i]);
+        if (e != cudaSuccess) return e;
+    }
+    return cudaSuccess;
+}
+
+cudaError_t set_attributes_layout(int num_sms) {
+    (void)num_sms;
+    static const void *const kKernels[] = {
+        (const void *)dsm_sum_kernel,
+        (const void *)nsm_sum_kernel,
+        (const void *)pax_sum_kernel};
+    const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
+    if (le != cudaSuccess) return le;
+    return cudaSuccess;
+}
+
 }  // namespace h2tap

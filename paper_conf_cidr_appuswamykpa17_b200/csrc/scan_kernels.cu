@@ -13,6 +13,7 @@
 
 #include "bulk_pipeline.cuh"
 #include "kernels.cuh"
+#include "peer.cuh"
 
 namespace h2tap {
 namespace {
@@ -689,14 +690,27 @@ __global__ void q1_compact_kernel(Q1Scratch g) {
     }
 }
 
-// Multi-GPU: fold gathered per-rank groups into the (clean) global table.
-__global__ void q1_merge_kernel(const Q1Group *__restrict__ all, uint64_t n, Q1Scratch g) {
-    const uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
-    if (i == 0) *g.ngroups = 0;
-    if (i < n) {
-        const Q1Group x = all[i];
-        q1_global_add(g, (1ull << 32) | (unsigned int)(int)x.key, (unsigned long long)x.cnt, x.qty,
-                      x.amt);
+// Multi-GPU (a7): every rank pushed its compacted group list into this rank's
+// mailbox (launch_peer_push) and launch_peer_wait saw all of them arrive; fold every list (this
+// rank's included) into the clean global table; q1_compact + q1_emit then run as on one GPU.
+__global__ void __launch_bounds__(256) q1_peer_merge_kernel(PeerArgs p, Q1Scratch g) {
+    pdl_wait();
+    pdl_trigger();
+    const unsigned long long s = peer::cur_seq(p);
+    if (blockIdx.x == 0 && threadIdx.x == 0) *g.ngroups = 0;
+    const int par = (int)(s & 1);
+    const unsigned long long stride = (unsigned long long)gridDim.x * blockDim.x;
+    for (int k = 0; k < p.world; ++k) {
+        const char *slot = peer::mbox(p, p.rank, par, k);
+        const unsigned long long n = *reinterpret_cast<const volatile unsigned long long *>(slot);
+        const Q1Group *list = reinterpret_cast<const Q1Group *>(slot + 16);
+        for (unsigned long long i = (unsigned long long)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
+            // (.cg: peer-written data is read from L2, never from a possibly stale L1 line)
+            const longlong2 a = __ldcg(reinterpret_cast<const longlong2 *>(list + i));
+            const longlong2 b = __ldcg(reinterpret_cast<const longlong2 *>(list + i) + 1);
+            const Q1Group x{a.x, a.y, b.x, b.y};
+            q1_global_add(g, (1ull << 32) | (unsigned int)(int)x.key, (unsigned long long)x.cnt, x.qty, x.amt);
+        }
     }
 }
 
@@ -758,12 +772,6 @@ void launch_q6(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uin
 void launch_q6_tma(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uint64_t n,
                    int64_t d_lo, int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s,
                    int num_sms, cudaStream_t st) {
-    static bool init = false;
-    if (!init) {
-        cudaFuncSetAttribute(q6_tma_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                             (int)sizeof(Q6TmaSmem));
-        init = true;
-    }
     const uint64_t nchunks = (n + kQ6Chunk - 1) / kQ6Chunk;
     const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
     launch_pdl(q6_tma_kernel, grid, kTmaThreads, sizeof(Q6TmaSmem), st,
@@ -783,12 +791,6 @@ void launch_q1_reset(const Q1Scratch &s, cudaStream_t st) {
 void launch_q1(const int32_t *number, const int64_t *deliv, const int32_t *qty,
                const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int num_sms,
                cudaStream_t st) {
-    static bool init = false;
-    if (!init) {
-        cudaFuncSetAttribute(q1_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                             (int)sizeof(Q1Smem));
-        init = true;
-    }
     uint64_t want = ((n >> 2) + kQ1Threads - 1) / kQ1Threads;
     uint64_t grid = (uint64_t)num_sms * 2;
     if (want < grid) grid = want ? want : 1;
@@ -804,11 +806,6 @@ void launch_q1_tma(const int32_t *number, const int64_t *deliv, const int32_t *q
                    cudaStream_t st) {
     using Cfg = Q1TmaCfg<false>;
     const size_t smem = sizeof(Q1StagesT<Cfg::kS>) + sizeof(Q1SmemT<Cfg::kT>);
-    static bool init = false;
-    if (!init) {
-        cudaFuncSetAttribute(q1_tma_kernel<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        init = true;
-    }
     const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
     const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
     launch_pdl(q1_tma_kernel<false>, grid, (Q1TmaCfg<false>::kW + 1) * 32, smem, st, number, reinterpret_cast<const long long *>(deliv), qty,
@@ -823,11 +820,6 @@ void launch_q61_tma(const int32_t *number, const int64_t *deliv, const int32_t *
                     cudaStream_t st) {
     using Cfg = Q1TmaCfg<true>;
     const size_t smem = sizeof(Q1StagesT<Cfg::kS>) + sizeof(Q1SmemT<Cfg::kT>);
-    static bool init = false;
-    if (!init) {
-        cudaFuncSetAttribute(q1_tma_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        init = true;
-    }
     const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
     const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
     launch_pdl(q1_tma_kernel<true>, grid, kQ61Threads, smem, st, number, reinterpret_cast<const long long *>(deliv),
@@ -841,14 +833,53 @@ void launch_q1_compact(const Q1Scratch &s, cudaStream_t st) {
     count_launches(1);
 }
 
-void launch_q1_merge(const Q1Group *all, uint64_t n, const Q1Scratch &s, cudaStream_t st) {
-    q1_merge_kernel<<<(unsigned)((n + 255) / 256 + 1), 256, 0, st>>>(all, n, s);
+void launch_q1_peer_merge(const PeerArgs &p, const Q1Scratch &s, int num_sms, cudaStream_t st) {
+    launch_pdl(q1_peer_merge_kernel, (unsigned)num_sms, 256, 0, st, p, s);
     count_launches(1);
 }
 
 void launch_q1_emit(const Q1Scratch &s, uint64_t max_groups, cudaStream_t st) {
     launch_pdl(q1_emit_kernel, (unsigned)((max_groups + 255) / 256), 256, 0, st, s);
     count_launches(1);
+}
+
+// Load every kernel of this file now (CUDA lazy loading would otherwise load a kernel at its first
+// launch, which waits for the device to idle — with N logical ranks on one device, behind another
+// rank's kernel that is waiting for this rank: a deadlock).
+static cudaError_t force_load(const void *const *fs, size_t n) {
+    for (size_t i = 0; i < n; ++i) {
+        cudaFuncAttributes a;
+        const cudaError_t e = cudaFuncGetAttributes(&a, fs[i]);
+        if (e != cudaSuccess) return e;
+    }
+    return cudaSuccess;
+}
+
+cudaError_t set_attributes_scan(int num_sms) {
+    static const void *const kKernels[] = {
+        (const void *)q1_compact_kernel,
+        (const void *)q1_emit_kernel,
+        (const void *)q1_kernel,
+        (const void *)q1_peer_merge_kernel,
+        (const void *)q1_tma_kernel<false>,
+        (const void *)q1_tma_kernel<true>,
+        (const void *)q6_kernel,
+        (const void *)q6_tma_kernel};
+    const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
+    if (le != cudaSuccess) return le;
+
+    (void)num_sms;
+    cudaError_t e = cudaFuncSetAttribute(q6_tma_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                         (int)sizeof(Q6TmaSmem));
+    if (e == cudaSuccess)
+        e = cudaFuncSetAttribute(q1_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(Q1Smem));
+    if (e == cudaSuccess)
+        e = cudaFuncSetAttribute(q1_tma_kernel<false>, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                 (int)(sizeof(Q1StagesT<Q1TmaCfg<false>::kS>) + sizeof(Q1SmemT<Q1TmaCfg<false>::kT>)));
+    if (e == cudaSuccess)
+        e = cudaFuncSetAttribute(q1_tma_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                 (int)(sizeof(Q1StagesT<Q1TmaCfg<true>::kS>) + sizeof(Q1SmemT<Q1TmaCfg<true>::kT>)));
+    return e;
 }
 
 }  // namespace h2tap

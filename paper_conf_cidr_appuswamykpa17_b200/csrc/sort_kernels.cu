@@ -21,6 +21,7 @@
 
 #include "cache_hints.cuh"
 #include "kernels.cuh"
+#include "peer.cuh"
 
 namespace h2tap {
 namespace {
@@ -312,14 +313,16 @@ __global__ void permute_kernel(const Q18Row *__restrict__ rows, const long long 
 
 __device__ __forceinline__ int bitwidth_dev(unsigned long long x) { return x ? 64 - __clzll(x) : 0; }
 
-__device__ Q18Plan make_q18_plan(const Q18Stats *__restrict__ stats, const Q18Zone &z,
-                                 const unsigned long long *nout, int bucket_bits, int allow_carry,
-                                 unsigned int *flag) {
-    const Q18Stats st = *stats;
+// The plan from the statistics: `n_spec` rows decide whether there is anything to order (one
+// GPU: > 1 rows, the single-row case takes the row-id path; distributed: >= 1 row anywhere, the
+// spec must be filled on every rank so that a lone row's carry record decodes).
+__device__ Q18Plan make_q18_plan_vals(const Q18Stats &st, const Q18Zone &z, unsigned long long n_local,
+                                      bool fill_spec, int bucket_bits, int allow_carry, unsigned int *flag) {
     Q18Plan p{};
-    p.n = *nout;
+    p.n = n_local;
+    p.bucket_bits = bucket_bits;
     Q18SortSpec &sp = p.spec;
-    if (p.n > 1) {
+    if (fill_spec) {
         sp.amt_max = st.amt_max;
         sp.ent_min = st.ent_min;
         sp.w_min = z.w_min; sp.d_min = z.d_min; sp.o_min = z.o_min;
@@ -344,6 +347,13 @@ __device__ Q18Plan make_q18_plan(const Q18Stats *__restrict__ stats, const Q18Zo
         p.shift = sp.prefix_bits > bucket_bits ? sp.prefix_bits - bucket_bits : 0;
     }
     return p;
+}
+
+__device__ Q18Plan make_q18_plan(const Q18Stats *__restrict__ stats, const Q18Zone &z,
+                                 const unsigned long long *nout, int bucket_bits, int allow_carry,
+                                 unsigned int *flag) {
+    const unsigned long long n = *nout;
+    return make_q18_plan_vals(*stats, z, n, n > 1, bucket_bits, allow_carry, flag);
 }
 
 // One thread: the ORDER BY plan from the HAVING statistics (amount_sum, o_entry_d) and the
@@ -603,7 +613,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
 #pragma unroll
         for (int u = 0; u < kPre; ++u) {
             const unsigned int i = threadIdx.x + u * kEmThreads;
-            if (i < m) pre[u] = __ldcs(kv + lo + i);
+            if (i < m) pre[u] = __ldcg(kv + lo + i);
         }
     };
     for (unsigned int i = threadIdx.x; i <= kLsSubMax; i += kEmThreads) S.sub[i] = 0;
@@ -629,7 +639,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
             }
         }
         for (unsigned int i = threadIdx.x + kPre * kEmThreads; i < m; i += kEmThreads) {  // rest
-            const ulonglong2 r = __ldcs(kv + lo + i);
+            const ulonglong2 r = __ldcg(kv + lo + i);
             S.rec[i] = r;
             atomicAdd(&S.sub[(unsigned int)(r.x >> ssh) & smask], 1u);
         }
@@ -735,10 +745,17 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
                          const unsigned int *__restrict__ offset, int nb,
                          const Q18Plan *__restrict__ plan, const Q18Row *__restrict__ rows,
                          const long long *__restrict__ amt, Q18Cols dst, unsigned int *flag,
-                         unsigned int *big, int sub_log2 = 3) {
+                         unsigned int *big, int sub_log2 = 3, PeerArgs pa = PeerArgs{}) {
     pdl_wait();
     pdl_trigger();
     extern __shared__ __align__(16) unsigned char smem_raw[];
+    if (pa.world > 1) {  // distributed ORDER BY: this rank's buckets, exchanged into its heap
+        // (their arrival was awaited by the one-thread peer_wait launched before this grid)
+        const unsigned long long xs = plan->xseq;
+        if (plan->err & (kPeerErrHeap | kPeerErrOutCap | kPeerErrNoCarry | kPeerErrTimeout)) return;
+        k = reinterpret_cast<const unsigned long long *>(peer::heap(pa, pa.rank, (int)(xs & 1)));
+        nb = (int)plan->nb_mine;  // offset = the receive offsets of those buckets
+    }
     if (kPairs && plan->spec.carry) {  // uniform: the whole ORDER BY runs on carry records
         carry_sort_emit<(kMin > 0 ? kLcCapLarge : kLsCap), kMin>(
             reinterpret_cast<const ulonglong2 *>(k), offset, nb, plan, dst, flag, big, smem_raw, sub_log2);
@@ -975,6 +992,7 @@ ob_hist_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ am
     const uint64_t n = P.n;
     const Q18SortSpec sp = P.spec;
     const int shift = P.shift;
+    if (P.dist) nb = 1 << P.bucket_bits;  // distributed: from the global row count (<= launch nb)
     const bool amt_only = sp.bits_a > 0 && shift >= sp.prefix_bits - sp.bits_a;
     for (int i = threadIdx.x; i < nb; i += kObThreads) h[i] = 0;
     __syncthreads();
@@ -1003,9 +1021,10 @@ ob_hist_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ am
 constexpr int kScanWarps = 32;
 __global__ void __launch_bounds__(32 * kScanWarps)
 ob_scan_kernel(unsigned int *__restrict__ mat, int G, int nb, unsigned int *__restrict__ count,
-               unsigned int *__restrict__ offset, unsigned int *ticket) {
+               unsigned int *__restrict__ offset, unsigned int *ticket, const Q18Plan *__restrict__ plan) {
     pdl_wait();
     pdl_trigger();
+    if (plan && plan->dist) nb = 1 << plan->bucket_bits;  // (grid sized for the launch nb)
     extern __shared__ unsigned int tile[];  // [G][32]; the last block reuses it for nb totals
     __shared__ bool last;
     __shared__ unsigned int tot[kScanWarps][32];
@@ -1084,6 +1103,7 @@ ob_scatter_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__
     const uint64_t n = plan->n;
     const Q18SortSpec sp = plan->spec;
     const int shift = plan->shift;
+    if (plan->dist) nb = 1 << plan->bucket_bits;
     const unsigned int *row = mat + (uint64_t)blockIdx.x * nb;
     for (int i = threadIdx.x; i < nb; i += kObThreads) cur[i] = offset[i] + row[i];
     __syncthreads();
@@ -1125,18 +1145,6 @@ void q18_bucket_order(const Q18Row *rows, const long long *amt, const Q18Plan *p
     auto end = [&] { if (marks) marks->end(); };
     if (bucket_bits > kBucketMaxBits) bucket_bits = kBucketMaxBits;
     const int nb = 1 << bucket_bits;
-    static bool init = false;
-    if (!init) {
-        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapSmall, 0>,
-                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapSmall>));
-        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall>,
-                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(LsSmem<kLsCapLarge>));
-        cudaFuncSetAttribute(q18_keys_hist_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                             4 << kBucketMaxBits);
-        cudaFuncSetAttribute(bucket_scatter_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                             4 << kBucketMaxBits);
-        init = true;
-    }
     cudaMemsetAsync(s.count, 0, sizeof(unsigned int) * (nb + 1), st);
     cudaMemsetAsync(s.big, 0, sizeof(unsigned int), st);
     const uint64_t n1 = n_max ? n_max : 1;
@@ -1194,18 +1202,6 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, Q18Plan *plan
     if (bucket_bits > kBucketMaxBits) bucket_bits = kBucketMaxBits;
     const int nb = 1 << bucket_bits;
     const int G = ob_grid(num_sms);
-    static bool init = false;
-    if (!init) {
-        cudaFuncSetAttribute(bucket_local_emit_kernel<kObCap, 0, true>,
-                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kObSmem);
-        cudaFuncSetAttribute(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>,
-                             cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kObSmemLarge);
-        cudaFuncSetAttribute(ob_hist_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 << kBucketMaxBits);
-        cudaFuncSetAttribute(ob_scatter_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 << kBucketMaxBits);
-        cudaFuncSetAttribute(ob_scan_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                             4 * std::max(32 * G, 1 << kBucketMaxBits));
-        init = true;
-    }
     (void)n_max;
     // carry sort: ~2^sub_log2 rows per sub-bucket (rank loop vs sub-bucket scan; knob for A/B)
     static const int sub_log2 = [] {
@@ -1220,7 +1216,7 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, Q18Plan *plan
     end();
     begin("q18_sort_scan");
     launch_pdl(ob_scan_kernel, (nb + 31) / 32, 32 * kScanWarps, 4 * std::max(32 * G, nb), st, s.mat, G, nb, s.count,
-                                                                                   s.offset, s.ticket);
+               s.offset, s.ticket, (const Q18Plan *)plan);
     count_launches(1);
     end();
     begin("q18_bucket_scatter");
@@ -1231,14 +1227,366 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, Q18Plan *plan
     begin("q18_bucket_sort_emit");
     const unsigned lb = (unsigned)nb < (unsigned)num_sms * 6 ? (unsigned)nb : (unsigned)num_sms * 6;
     launch_pdl(bucket_local_emit_kernel<kObCap, 0, true>, lb, kEmThreads, kObSmem, st,
-        s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2);
+        s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2, PeerArgs{});
     count_launches(1);
     end();
     begin("q18_bucket_sort_emit_large");
     launch_pdl(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>, (unsigned)num_sms, kEmThreads, kObSmemLarge, st,
-        s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2);
+        s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2, PeerArgs{});
     count_launches(1);
     end();
+}
+
+}  // namespace h2tap
+
+// ==================================== distributed ORDER BY (world > 1) ===
+// Q18 groups are warehouse-local (every join predicate has w_id equality), so each rank computes
+// its groups alone; only the ORDER BY crosses ranks. The result is range-partitioned: the buckets
+// of the carry-record sort (top bits of the exact composite key, one definition on every rank)
+// are assigned to ranks by their GLOBAL row positions, so rank k ends up holding rows
+// [row0_k, row0_k + n_k) of the globally ordered result, ~1/world of it, sorted by the same
+// per-bucket shared-memory sort as on one GPU. No rank gathers or re-sorts anyone else's rows.
+//   meta  (1 warp):  push {nout, err, stats, zone} -> every rank; wait; reduce; derive the plan
+//                    (widths from the GLOBAL min/max, bucket bits from the global row count)
+//   hist + scan:     as on one GPU, over this rank's rows (local bucket counts and offsets)
+//   push counts:     launch_peer_push of the nb local bucket counts
+//   route (1 block): wait; per bucket the total over ranks and this rank's prefix among them;
+//                    scan -> global start; owner = the rank whose 1/world slice the start is in;
+//                    the destination position of this rank's records of every bucket; the receive
+//                    offsets of this rank's own buckets; heap / output capacity checks
+//   scatter:         as on one GPU: the carry records in local bucket order
+//   send:            per bucket, one warp copies this rank's records (contiguous, 16 B each) to
+//                    its place in the owner's heap over NVLink; the last block signals every rank
+//   emit:            as on one GPU over this rank's buckets, reading the records from its heap
+namespace h2tap {
+namespace {
+using namespace peer;
+
+struct Q18Meta {                 // one rank's contribution to the plan (mailbox payload)
+    unsigned long long nout;
+    unsigned int err, pad;
+    Q18Stats st;
+    Q18Zone z;
+};
+
+__global__ void q18_dist_meta_kernel(PeerArgs p, const unsigned long long *nout, const unsigned int *err,
+                                     const Q18Stats *stats, Q18Zone zone, int allow_carry, int nb_max_bits,
+                                     Q18Plan *plan, unsigned int *flag) {
+    pdl_wait();
+    trigger_before_wait(p);
+    if (threadIdx.x != 0) return;  // (a CTA triggers when one of its threads does: thread 0 below)
+    const unsigned long long s = next_seq(p);
+    const int par = (int)(s & 1);
+    Q18Meta m{};
+    m.nout = *nout;
+    m.err = *err;
+    m.st = *stats;
+    m.z = zone;
+    for (int k = 0; k < p.world; ++k) *reinterpret_cast<Q18Meta *>(mbox(p, k, par, p.rank)) = m;
+    signal_all(p, s);
+    Q18Meta g{};
+    g.st.amt_min = INT64_MAX; g.st.amt_max = INT64_MIN; g.st.ent_min = INT64_MAX; g.st.ent_max = INT64_MIN;
+    g.z = zone;
+    unsigned int perr = 0;
+    const bool ok = wait_all(p, s);
+    trigger_after_wait(p);
+    if (!ok) perr |= kPeerErrTimeout;
+    else
+        for (int k = 0; k < p.world; ++k) {
+            Q18Meta x;
+            const unsigned long long *src = reinterpret_cast<const unsigned long long *>(mbox(p, p.rank, par, k));
+            unsigned long long *dst = reinterpret_cast<unsigned long long *>(&x);
+            for (int q = 0; q < (int)(sizeof(Q18Meta) / 8); ++q) dst[q] = __ldcg(src + q);
+            g.nout += x.nout;
+            g.err |= x.err;
+            if (x.nout) {  // a rank without result rows has sentinel statistics: skip them
+                g.st.amt_min = min(g.st.amt_min, x.st.amt_min); g.st.amt_max = max(g.st.amt_max, x.st.amt_max);
+                g.st.ent_min = min(g.st.ent_min, x.st.ent_min); g.st.ent_max = max(g.st.ent_max, x.st.ent_max);
+            }
+            int *gz = reinterpret_cast<int *>(&g.z);
+            const int *xz = reinterpret_cast<const int *>(&x.z);
+            for (int q = 0; q < 6; ++q) { gz[2 * q] = min(gz[2 * q], xz[2 * q]); gz[2 * q + 1] = max(gz[2 * q + 1], xz[2 * q + 1]); }
+        }
+    // bucket bits from the global row count (~256-512 rows per bucket, as on one GPU)
+    int bb = 1;
+    while (bb < nb_max_bits && (g.nout >> (bb + 9)) > 0) ++bb;
+    Q18Plan P = make_q18_plan_vals(g.st, g.z, m.nout, g.nout >= 1, bb, allow_carry, flag);
+    P.dist = 1;
+    P.nbuckets = 1ull << bb;
+    P.n_total = g.nout;
+    P.err = g.err | perr;
+    if (g.nout >= 1 && !P.spec.carry) P.err |= kPeerErrNoCarry;  // the exchange moves carry records
+    if (P.err) P.n = 0;  // nothing is scattered; every rank reports the error
+    *plan = P;
+}
+
+// Receive-side plan (one block of 1024 threads; shared memory: nb totals). `count`/`offset` are
+// this rank's bucket counts / exclusive offsets (ob_scan); the mailboxes hold every rank's counts.
+constexpr int kRouteThreads = 1024;
+__global__ void __launch_bounds__(kRouteThreads)
+q18_dist_route_kernel(PeerArgs p, Q18Plan *plan, unsigned long long *__restrict__ send,
+                      unsigned int *__restrict__ recv_off, unsigned long long out_cap) {
+    pdl_wait();
+    trigger_before_wait(p);
+    extern __shared__ unsigned int tot[];          // [nb] totals -> global starts (exclusive)
+    __shared__ unsigned int wsum[kRouteThreads / 32];
+    __shared__ unsigned int lo[kMaxRanks + 1];     // first bucket of each rank (nb: none)
+    __shared__ int ok;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const unsigned long long s = cur_seq(p);       // the counts' push
+    if (threadIdx.x == 0) ok = wait_all(p, s) ? 1 : 0;
+    __syncthreads();
+    trigger_after_wait(p);
+    const int nb = 1 << plan->bucket_bits;
+    const int par = (int)(s & 1);
+    unsigned int perr = ok ? 0u : kPeerErrTimeout;
+    if (ok) {
+        for (int b = threadIdx.x; b < nb; b += kRouteThreads) {
+            unsigned int t = 0, pre = 0;
+            for (int k = 0; k < p.world; ++k) {
+                const unsigned int c = __ldcg(reinterpret_cast<const unsigned int *>(mbox(p, p.rank, par, k) + 16) + b);
+                t += c;
+                if (k < p.rank) pre += c;
+            }
+            tot[b] = t;
+            send[b] = pre;  // this rank's place among the bucket's ranks (completed below)
+        }
+    }
+    if (threadIdx.x <= kMaxRanks) lo[threadIdx.x] = (unsigned int)nb;
+    __syncthreads();
+    // exclusive scan of tot[]: each warp a contiguous span, warp-cooperative
+    const int span = (nb + kRouteThreads / 32 - 1) / (kRouteThreads / 32);
+    const int w0 = warp * span, w1 = min(nb, w0 + span);
+    unsigned int wt = 0;
+    for (int base = w0; base < w1; base += 32) {
+        const int i = base + lane;
+        wt += __reduce_add_sync(kFull, i < w1 ? tot[i] : 0u);
+    }
+    if (lane == 0) wsum[warp] = wt;
+    __syncthreads();
+    unsigned int acc = 0;
+    for (int w = 0; w < warp; ++w) acc += wsum[w];
+    for (int base = w0; base < w1; base += 32) {
+        const int i = base + lane;
+        const unsigned int c = i < w1 ? tot[i] : 0u;
+        unsigned int x = c;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const unsigned int y = __shfl_up_sync(kFull, x, o);
+            if (lane >= o) x += y;
+        }
+        if (i < w1) tot[i] = acc + x - c;
+        acc += __shfl_sync(kFull, x, 31);
+    }
+    __syncthreads();
+    unsigned long long T = 0;
+    for (int w = 0; w < kRouteThreads / 32; ++w) T += wsum[w];
+    const int W = p.world;
+    auto owner = [&](int b) -> int {
+        if (T == 0) return 0;
+        const unsigned long long o = (unsigned long long)tot[b] * (unsigned long long)W / T;
+        return o >= (unsigned long long)W ? W - 1 : (int)o;
+    };
+    // lo[k] = first bucket owned by a rank >= k (owners are non-decreasing in b)
+    for (int b = threadIdx.x; b < nb; b += kRouteThreads) {
+        const int o = owner(b), op = b ? owner(b - 1) : -1;
+        for (int k = op + 1; k <= o; ++k) lo[k] = (unsigned int)b;
+    }
+    __syncthreads();
+    auto row0 = [&](int k) -> unsigned long long { return lo[k] < (unsigned int)nb ? tot[lo[k]] : T; };
+    for (int b = threadIdx.x; b < nb; b += kRouteThreads) {
+        const int o = owner(b);
+        const unsigned long long pos = (unsigned long long)tot[b] - row0(o) + send[b];
+        send[b] = ((unsigned long long)o << 56) | pos;
+    }
+    const unsigned int b_lo = lo[p.rank], b_hi = lo[p.rank + 1] < lo[p.rank] ? lo[p.rank] : lo[p.rank + 1];
+    const unsigned long long r0 = row0(p.rank);
+    for (unsigned int b = b_lo + threadIdx.x; b <= b_hi; b += kRouteThreads)
+        recv_off[b - b_lo] = (unsigned int)((b < (unsigned int)nb ? (unsigned long long)tot[b] : T) - r0);
+    if (threadIdx.x == 0) {
+        unsigned long long worst = 0;
+        for (int k = 0; k < W; ++k) {
+            const unsigned long long nk = (k + 1 < W ? row0(k + 1) : T) - row0(k);
+            worst = nk > worst ? nk : worst;
+        }
+        const unsigned long long mine = (p.rank + 1 < W ? row0(p.rank + 1) : T) - r0;
+        if (worst * 16ull > p.heap_half) perr |= kPeerErrHeap;      // the same decision on every rank
+        if (mine > out_cap) perr |= kPeerErrOutCap;                 // local: re-emitted by the host
+        plan->b_lo = b_lo;
+        plan->nb_mine = b_hi - b_lo;
+        plan->n_mine = mine;
+        plan->row0 = r0;
+        plan->xseq = s + 1;
+        plan->err |= perr;
+    }
+}
+
+// One warp per bucket: this rank's records of bucket b (contiguous after the local scatter) to
+// their place in the owner's heap; the last block publishes the exchange to every rank.
+__global__ void __launch_bounds__(1024)
+q18_dist_send_kernel(PeerArgs p, const Q18Plan *__restrict__ plan, const ulonglong2 *__restrict__ kv,
+                     const unsigned int *__restrict__ offset, const unsigned long long *__restrict__ send) {
+    pdl_wait();
+    pdl_trigger();
+    const unsigned long long s = next_seq(p);
+    const int par = (int)(s & 1);
+    if (!(plan->err & kPeerErrHeap) && !(plan->err & kPeerErrTimeout)) {
+        const int nb = 1 << plan->bucket_bits;
+        const int lane = threadIdx.x & 31;
+        const int nw = (int)(gridDim.x * (blockDim.x >> 5));
+        for (int b = (int)(blockIdx.x * (blockDim.x >> 5) + (threadIdx.x >> 5)); b < nb; b += nw) {
+            const unsigned int lo = offset[b], c = offset[b + 1] - lo;
+            if (c == 0) continue;
+            const unsigned long long d = send[b];
+            ulonglong2 *dst = reinterpret_cast<ulonglong2 *>(heap(p, (int)(d >> 56), par)) + (d & ((1ull << 56) - 1));
+            for (unsigned int i = lane; i < c; i += 32) dst[i] = __ldcs(kv + lo + i);
+        }
+    }
+    if (block_done_last(p)) signal_all(p, s);
+}
+
+struct Q18SmallDist { unsigned long long nout; unsigned int err, tie; Q18Stats st; unsigned long long row0, n_total; };
+__global__ void q18_dist_publish_kernel(const Q18Plan *plan, const unsigned int *tie, Q18SmallDist *out) {
+    pdl_wait();
+    pdl_trigger();
+    out->nout = plan->n_mine;
+    out->err = plan->err;
+    out->tie = *tie;
+    out->row0 = plan->row0;
+    out->n_total = plan->n_total;
+}
+
+}  // namespace
+
+void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long long *amt, Q18Plan *plan,
+                           const Q18PlanArgs &meta, const unsigned int *err, const BucketSort &s,
+                           unsigned long long *send, unsigned int *recv_off, uint64_t out_cap,
+                           const Q18Cols &dst, unsigned int *flag, void *host_small, int num_sms,
+                           cudaStream_t st, PhaseMarks *marks) {
+    auto begin = [&](const char *nm) { if (marks) marks->begin(nm); };
+    auto end = [&] { if (marks) marks->end(); };
+    const int nb = 1 << kBucketMaxBits;  // launch sizes: the largest bucket count the plan may pick
+    const int G = ob_grid(num_sms);
+    begin("q18_dist_meta");
+    launch_pdl(q18_dist_meta_kernel, 1, 32, 0, st, pa, meta.nout, err, meta.stats, meta.zone, meta.allow_carry,
+               kBucketMaxBits, plan, flag);
+    count_launches(1);
+    end();
+    begin("q18_sort_hist");
+    launch_pdl(ob_hist_kernel, G, kObThreads, nb * 4, st, rows, amt, plan, nb, s.mat, s.big, 0, Q18PlanArgs{}, 0, flag);
+    count_launches(1);
+    end();
+    begin("q18_sort_scan");
+    launch_pdl(ob_scan_kernel, (nb + 31) / 32, 32 * kScanWarps, 4 * std::max(32 * G, nb), st, s.mat, G, nb, s.count,
+               s.offset, s.ticket, (const Q18Plan *)plan);
+    count_launches(1);
+    end();
+    begin("q18_dist_counts");
+    launch_peer_push(pa, s.count, &plan->nbuckets, 0, 4u, num_sms, st);
+    end();
+    begin("q18_dist_route");
+    launch_pdl(q18_dist_route_kernel, 1, kRouteThreads, 4 * nb, st, pa, plan, send, recv_off,
+               (unsigned long long)out_cap);
+    count_launches(1);
+    end();
+    begin("q18_bucket_scatter");
+    launch_pdl(ob_scatter_kernel, G, kObThreads, nb * 4, st, rows, amt, (const Q18Plan *)plan, nb, (const unsigned int *)s.mat,
+               (const unsigned int *)s.offset, s.kv);
+    count_launches(1);
+    end();
+    begin("q18_dist_send");
+    launch_pdl(q18_dist_send_kernel, (unsigned)num_sms, 1024, 0, st, pa, (const Q18Plan *)plan,
+               reinterpret_cast<const ulonglong2 *>(s.kv), (const unsigned int *)s.offset, (const unsigned long long *)send);
+    count_launches(1);
+    end();
+    begin("q18_dist_wait");
+    launch_peer_wait(pa, st);
+    end();
+    q18_dist_emit(pa, plan, recv_off, dst, flag, s, num_sms, st, marks);
+    launch_pdl(q18_dist_publish_kernel, 1, 1, 0, st, (const Q18Plan *)plan, (const unsigned int *)flag,
+               static_cast<Q18SmallDist *>(host_small));
+    count_launches(1);
+}
+
+void q18_dist_emit(const PeerArgs &pa, const Q18Plan *plan, const unsigned int *recv_off, const Q18Cols &dst,
+                   unsigned int *flag, const BucketSort &s, int num_sms, cudaStream_t st, PhaseMarks *marks) {
+    auto begin = [&](const char *nm) { if (marks) marks->begin(nm); };
+    auto end = [&] { if (marks) marks->end(); };
+    static const int sub_log2 = [] {
+        const char *v = std::getenv("H2TAP_SUB_ROWS_LOG2");
+        return v ? std::max(0, std::min(6, std::atoi(v))) : 1;
+    }();
+    // the emit walks at most 2^kBucketMaxBits buckets; the grid covers the SMs
+    begin("q18_bucket_sort_emit");
+    launch_pdl(bucket_local_emit_kernel<kObCap, 0, true>, (unsigned)num_sms * 6, kEmThreads, kObSmem, st,
+               (const unsigned long long *)nullptr, (const unsigned int *)nullptr, recv_off, 0, plan,
+               (const Q18Row *)nullptr, (const long long *)nullptr, dst, flag, s.big, sub_log2, pa);
+    count_launches(1);
+    end();
+    begin("q18_bucket_sort_emit_large");
+    launch_pdl(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>, (unsigned)num_sms, kEmThreads, kObSmemLarge, st,
+               (const unsigned long long *)nullptr, (const unsigned int *)nullptr, recv_off, 0, plan,
+               (const Q18Row *)nullptr, (const long long *)nullptr, dst, flag, s.big, sub_log2, pa);
+    count_launches(1);
+    end();
+}
+
+// Dynamic shared-memory limits of every ORDER BY kernel, set once per device (h2tap_open).
+// Load every kernel of this file now (CUDA lazy loading would otherwise load a kernel at its first
+// launch, which waits for the device to idle — with N logical ranks on one device, behind another
+// rank's kernel that is waiting for this rank: a deadlock).
+static cudaError_t force_load(const void *const *fs, size_t n) {
+    for (size_t i = 0; i < n; ++i) {
+        cudaFuncAttributes a;
+        const cudaError_t e = cudaFuncGetAttributes(&a, fs[i]);
+        if (e != cudaSuccess) return e;
+    }
+    return cudaSuccess;
+}
+
+cudaError_t set_attributes_sort(int num_sms) {
+    static const void *const kKernels[] = {
+        (const void *)bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall>,
+        (const void *)bucket_local_emit_kernel<kLsCapLarge, kObCap, true>,
+        (const void *)bucket_local_emit_kernel<kLsCapSmall, 0>,
+        (const void *)bucket_local_emit_kernel<kObCap, 0, true>,
+        (const void *)bucket_scatter_kernel,
+        (const void *)digit_scan_kernel,
+        (const void *)field_keys_kernel,
+        (const void *)hist_kernel,
+        (const void *)iota_kernel,
+        (const void *)ob_hist_kernel,
+        (const void *)ob_scan_kernel,
+        (const void *)ob_scatter_kernel,
+        (const void *)permute_kernel,
+        (const void *)q18_dist_meta_kernel,
+        (const void *)q18_dist_publish_kernel,
+        (const void *)q18_dist_route_kernel,
+        (const void *)q18_dist_send_kernel,
+        (const void *)q18_keys_hist_kernel,
+        (const void *)q18_plan_kernel,
+        (const void *)scatter_kernel};
+    const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
+    if (le != cudaSuccess) return le;
+
+    const int G = ob_grid(num_sms);
+    const struct { const void *f; int bytes; } a[] = {
+        {(const void *)bucket_local_emit_kernel<kLsCapSmall, 0>, (int)sizeof(LsSmem<kLsCapSmall>)},
+        {(const void *)bucket_local_emit_kernel<kLsCapLarge, kLsCapSmall>, (int)sizeof(LsSmem<kLsCapLarge>)},
+        {(const void *)q18_keys_hist_kernel, 4 << kBucketMaxBits},
+        {(const void *)bucket_scatter_kernel, 4 << kBucketMaxBits},
+        {(const void *)bucket_local_emit_kernel<kObCap, 0, true>, (int)kObSmem},
+        {(const void *)bucket_local_emit_kernel<kLsCapLarge, kObCap, true>, (int)kObSmemLarge},
+        {(const void *)ob_hist_kernel, 4 << kBucketMaxBits},
+        {(const void *)ob_scatter_kernel, 4 << kBucketMaxBits},
+        {(const void *)ob_scan_kernel, 4 * std::max(32 * G, 1 << kBucketMaxBits)},
+        {(const void *)q18_dist_route_kernel, 4 << kBucketMaxBits},
+    };
+    for (const auto &x : a) {
+        const cudaError_t e = cudaFuncSetAttribute(x.f, cudaFuncAttributeMaxDynamicSharedMemorySize, x.bytes);
+        if (e != cudaSuccess) return e;
+    }
+    return cudaSuccess;
 }
 
 }  // namespace h2tap

@@ -167,4 +167,31 @@ void launch_minmax_i32(const int32_t *p, uint64_t n, int *out, int num_sms, cuda
     minmax_kernel<<<(unsigned)blocks, 256, 0, st>>>(p, n, out);
 }
 
+// Load every kernel of this file now (CUDA lazy loading would otherwise load a kernel at its first
+// launch, which waits for the device to idle — with N logical ranks on one device, behind another
+// rank's kernel that is waiting for this rank: a deadlock).
+static cudaError_t force_load(const void *const *fs, size_t n) {
+    for (size_t i = 0; i < n; ++i) {
+        cudaFuncAttributes a;
+        const cudaError_t e = cudaFuncGetAttributes(&a, fs[i]);
+        if (e != cudaSuccess) return e;
+    }
+    return cudaSuccess;
+}
+
+cudaError_t set_attributes_store(int num_sms) {
+    (void)num_sms;
+    static const void *const kKernels[] = {
+        (const void *)apply_updates_kernel<int32_t>,
+        (const void *)apply_updates_kernel<int64_t>,
+        (const void *)cow_catchup_kernel<4>,
+        (const void *)cow_catchup_kernel<8>,
+        (const void *)gate_kernel,
+        (const void *)minmax_kernel,
+        (const void *)stats_init_kernel};
+    const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
+    if (le != cudaSuccess) return le;
+    return cudaSuccess;
+}
+
 }  // namespace h2tap
