@@ -7,16 +7,20 @@ group-join, HAVING compaction, customer probe, ORDER BY) through the C ABI, each
 cross-GPU merge when N > 1. Workload = BASELINE.json configs[1]/[2]: W = 100 TPC-C warehouses
 per GPU (~30M order_line rows), synthetic ('spread' population, seed 1).
 
-value  = order_line rows processed per second by the step's three queries, whole job
-         (3 x visible order_line rows x N / step time), snapshot resident in HBM.
+value  = order_line rows per second through one full pass of the hot path, whole job: every
+         rank's visible order_line rows (each counted ONCE per step, although Q6, Q1 and Q18 all
+         read them) / step time (max over ranks), snapshot resident in HBM.
 e2e    = same metric through the public API with host buffers: each step refreshes the snapshot
-         from pinned host memory (full reload, H2D inside the timed region) and returns every
-         result to host memory.
+         from pinned host memory (full reload, H2D inside the timed region), runs the batch and
+         returns every result to host memory; the serial figure (queries read that step's upload).
 roofline: the dominant kernel's algorithmic bytes per launch / its CUDA-event duration,
-         against MEASURED_PEAKS.json hbm_gbs.
+         against MEASURED_PEAKS.json hbm_gbs (copy) and the live read-stream peak.
+c1     = BASELINE configs[0]: Q6 at W=1 on one GPU, device and e2e latency, oracle beside it.
 
 Usage: python bench.py [--gpus N --steps K --warmup W] [--impl ours|reference]
-       torchrun --nproc-per-node N bench.py --gpus N ...
+       [--total-warehouses T]   (strong scaling: T warehouses split over the N GPUs, config C4)
+With --gpus N > 1 and no torchrun environment, bench.py launches its N ranks itself
+(torch.distributed.run, 127.0.0.1); under torchrun WORLD_SIZE must equal --gpus.
 """
 from __future__ import annotations
 
@@ -50,6 +54,10 @@ def parse():
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
     ap.add_argument("--warehouses", type=int, default=100, help="warehouses per GPU (weak scaling)")
+    ap.add_argument("--total-warehouses", type=int, default=None,
+                    help="strong scaling: this many warehouses split over the GPUs (config C4)")
+    ap.add_argument("--peer-heap-mb", type=int, default=0, help="world > 1: peer heap per rank (0 = 1 GiB)")
+    ap.add_argument("--no-c1", action="store_true", help="skip the config C1 line (Q6 at W=1)")
     ap.add_argument("--mode", default="spread", choices=["spread", "strict"])
     ap.add_argument("--e2e-steps", type=int, default=None)
     ap.add_argument("--no-cpu-baseline", action="store_true")
@@ -63,6 +71,57 @@ def dist_env():
     world = int(os.environ.get("WORLD_SIZE", "1"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
     return rank, world, local
+
+
+def spawn_ranks(a):
+    """--gpus N > 1 outside torchrun: launch the N ranks here (one process per GPU)."""
+    import socket
+    import torch
+    have = torch.cuda.device_count()
+    if have < a.gpus:
+        print(json.dumps({"error": f"--gpus {a.gpus} but {have} CUDA device(s) visible"}), flush=True)
+        return 2
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={a.gpus}",
+           "--master-addr=127.0.0.1", f"--master-port={port}", os.path.abspath(__file__)] + sys.argv[1:]
+    return subprocess.call(cmd)
+
+
+def host_cpu():
+    model = "unknown"
+    try:
+        for line in open("/proc/cpuinfo"):
+            if line.startswith("model name"):
+                model = line.split(":", 1)[1].strip()
+                break
+    except OSError:
+        pass
+    return {"nproc": os.cpu_count(), "cpu_model": model}
+
+
+class pinned_core:
+    """Run the oracle on one host core (taskset -c 1 equivalent: sched_setaffinity)."""
+
+    def __init__(self, core=1):
+        self.core = core
+        self.old = None
+
+    def __enter__(self):
+        try:
+            self.old = os.sched_getaffinity(0)
+            core = self.core if self.core in self.old else min(self.old)
+            os.sched_setaffinity(0, {core})
+            self.used = core
+        except (AttributeError, OSError):
+            self.used = None
+        return self
+
+    def __exit__(self, *exc):
+        if self.old:
+            os.sched_setaffinity(0, self.old)
 
 
 class Clocks:
@@ -168,16 +227,18 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None):
 
 # ------------------------------------------------------------------ reference --
 def cpu_oracle_sample(w_lo, sample_w, mode):
-    """Oracle (single-threaded C, as it stands) on a bounded sample of the same workload."""
+    """Oracle (single-threaded C, as it stands) on a bounded sample of the same workload, on one
+    pinned host core."""
     import oracle
     t = chgen.generate(w_lo, w_lo + sample_w, seed=1, mode=mode)
     n = len(t["order_line"]["ol_w_id"])
-    t0 = time.perf_counter()
-    oracle.q6(t, *Q6_P)
-    oracle.q1(t, *Q1_P)
-    oracle.q18(t, *Q18_P)
-    dt = time.perf_counter() - t0
-    return 3 * n / dt, dt, n
+    with pinned_core(1) as pc:
+        t0 = time.perf_counter()
+        oracle.q6(t, *Q6_P)
+        oracle.q1(t, *Q1_P)
+        oracle.q18(t, *Q18_P)
+        dt = time.perf_counter() - t0
+    return n / dt, dt, n, pc.used
 
 
 def run_reference(a):
@@ -189,54 +250,154 @@ def run_reference(a):
     sample_w = 10
     t = chgen.generate(1, 1 + sample_w, seed=1, mode=a.mode)
     n = len(t["order_line"]["ol_w_id"])
-    for _ in range(a.warmup):
-        oracle.q6(t, *Q6_P); oracle.q1(t, *Q1_P); oracle.q18(t, *Q18_P)
-    t0 = time.perf_counter()
-    for _ in range(a.steps):
-        oracle.q6(t, *Q6_P); oracle.q1(t, *Q1_P); oracle.q18(t, *Q18_P)
-    dt = time.perf_counter() - t0
-    value = 3 * n * a.steps / dt
+    with pinned_core(1) as pc:
+        for _ in range(a.warmup):
+            oracle.q6(t, *Q6_P); oracle.q1(t, *Q1_P); oracle.q18(t, *Q18_P)
+        t0 = time.perf_counter()
+        for _ in range(a.steps):
+            oracle.q6(t, *Q6_P); oracle.q1(t, *Q1_P); oracle.q18(t, *Q18_P)
+        dt = time.perf_counter() - t0
+    value = n * a.steps / dt
     sample = (f"each step = oracle Q6+Q1+Q18 over W={sample_w} warehouses ({n} order_line rows, "
-              f"'{a.mode}', seed 1), single thread")
+              f"'{a.mode}', seed 1), single thread pinned to core {pc.used}")
     print(json.dumps({
         "impl": "reference", "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": a.gpus,
         "steps": a.steps, "warmup": a.warmup, "ms_per_step": dt / a.steps * 1e3,
         "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "int64",
         "data": "synthetic", "config": {"workload": f"CH Q6+Q1+Q18 per step, sample W={sample_w}",
-                                        "mode": a.mode},
-        "cpu_baseline": {"value": value, "unit": UNIT, "cores": 1, "kind": "oracle", "sample": sample},
+                                        "mode": a.mode, "rows_counted": ROWS_COUNTED},
+        "cpu_baseline": dict({"value": value, "unit": UNIT, "cores": 1, "kind": "oracle", "sample": sample,
+                              "pinned_core": pc.used}, **host_cpu()),
         "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }))
     return 0
 
 
+ROWS_COUNTED = ("each visible order_line row counted once per step; one step = CH Q6 + Q1 + Q18 "
+                "over the snapshot (all three read every order_line row)")
+
+
 # ----------------------------------------------------------------------- ours --
+def event_ms(stream, fn, reps, flush=None):
+    """Median CUDA-event time of fn() on `stream` over `reps` runs (L2 flushed before each)."""
+    import torch
+    out = []
+    for _ in range(reps):
+        if flush:
+            flush()
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record(stream)
+        fn()
+        b.record(stream)
+        b.synchronize()
+        out.append(a.elapsed_time(b))
+    return float(np.median(out))
+
+
+def read_stream_peak(h, eng, stream):
+    """Live read-only HBM stream rate: the library's DSM layout kernel (one int32 column, pure
+    coalesced reads, NEXT-3) over 4 GiB — the read ceiling next to the copy peak of MEASURED_PEAKS."""
+    import torch
+    n = 1 << 30
+    col = torch.ones(n, dtype=torch.int32, device="cuda")
+    torch.cuda.synchronize()
+    best = 0.0
+    for _ in range(5):
+        _, ms = h.h2tap_layout_sum(eng, col, h.H2TAP_DSM, n, 1, [0])
+        best = max(best, 4.0 * n / (ms / 1e3) / 1e9)
+    del col
+    torch.cuda.empty_cache()
+    return round(best, 1)
+
+
+def c1_line(h, a):
+    """BASELINE configs[0]: CH Q6 at W=1 (~300 k order_line rows, 6 MB) on one GPU vs the oracle:
+    device latency (CUDA events around the query on the resident snapshot), e2e latency (the W=1
+    Q6 columns uploaded from pinned host memory + the query + the result on the host) and the
+    oracle's latency on one pinned host core, medians."""
+    import torch
+    import oracle
+    t = chgen.generate(1, 2, seed=1, mode=a.mode)
+    n = len(t["order_line"]["ol_w_id"])
+    cols = {"order_line": {c: torch.from_numpy(t["order_line"][c]).pin_memory()
+                           for c in ("ol_delivery_d", "ol_quantity", "ol_amount")}}
+    e = h.h2tap_open(0)
+    try:
+        h.h2tap_load_snapshot(e, cols, 1)
+        stream = torch.cuda.ExternalStream(h.h2tap_compute_stream(e))
+        got = None
+
+        def q():
+            nonlocal got
+            r = h.h2tap_run_query(e, h.H2TAP_Q6, Q6_P, flags=h.H2TAP_RESULT_DEVICE)
+            got = r.nrows
+            h.h2tap_free(r)
+        for _ in range(20):
+            q()
+        dev_ms = event_ms(stream, q, 100)
+        epoch = [1]
+
+        def e2e():
+            epoch[0] += 1
+            h.h2tap_load_snapshot(e, cols, epoch[0])
+            r = h.h2tap_run_query(e, h.H2TAP_Q6, Q6_P)
+            v = r.to_numpy()
+            h.h2tap_free(r)
+            return v
+        for _ in range(5):
+            res = e2e()
+        e2e_ms = []
+        for _ in range(50):
+            t0 = time.perf_counter()
+            res = e2e()
+            e2e_ms.append((time.perf_counter() - t0) * 1e3)
+        want = oracle.q6(t, *Q6_P)
+        assert int(res["revenue"][0]) == want["revenue"] and int(res["count_rows"][0]) == want["count"]
+        ora = []
+        with pinned_core(1) as pc:
+            for _ in range(5):
+                t0 = time.perf_counter()
+                oracle.q6(t, *Q6_P)
+                ora.append((time.perf_counter() - t0) * 1e3)
+        dev, ee, om = dev_ms, float(np.median(e2e_ms)), float(np.median(ora))
+        return {"workload": "CH Q6 at W=1 (BASELINE configs[0]), 1 GPU, parity vs the oracle checked",
+                "order_line_rows": n, "device_ms": round(dev, 4), "device_rows_per_s": n / (dev / 1e3),
+                "e2e_ms": round(ee, 4), "e2e_rows_per_s": n / (ee / 1e3),
+                "e2e_how": "per run: full reload of the 3 Q6 columns (6 MB) from pinned host memory + "
+                           "h2tap_run_query + result on the host; host wall clock, median of 50",
+                "oracle_ms": round(om, 3), "oracle_rows_per_s": n / (om / 1e3), "oracle_cores": 1,
+                "oracle_pinned_core": pc.used,
+                "note": "6 MB is L2-resident and launch-bound; % of HBM is not meaningful here"}
+    finally:
+        h.h2tap_close(e)
+
+
 def main():
     a = parse()
     if a.impl == "reference":
         return run_reference(a)
+    rank, world, local = dist_env()
+    if "WORLD_SIZE" not in os.environ and a.gpus > 1:
+        return spawn_ranks(a)
+    if world != a.gpus:
+        print(json.dumps({"error": f"WORLD_SIZE={world} but --gpus {a.gpus}"}), flush=True)
+        return 2
     import torch
     import torch.distributed as dist
 
-    rank, world, local = dist_env()
-    if world != a.gpus:
-        a.gpus = world if world > 1 else a.gpus
     torch.cuda.set_device(local)
-    if world > 1:
+    if world > 1:  # plumbing only: peer-handle exchange, barriers, max-over-ranks timing
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
 
     import paper_conf_cidr_appuswamykpa17_b200 as h
 
-    # ---- engine + NCCL bootstrap (ncclUniqueId broadcast over the torch process group)
-    nccl_id = None
+    eng = h.h2tap_open(local, rank, world, a.peer_heap_mb << 20)
     if world > 1:
-        obj = [h.h2tap_nccl_unique_id() if rank == 0 else None]
-        dist.broadcast_object_list(obj, src=0)
-        nccl_id = obj[0]
-    eng = h.h2tap_open(local, rank, world, nccl_id)
+        h.connect_torch_group(eng)
 
-    # ---- this rank's warehouse shard (weak scaling: a.warehouses per GPU)
-    W = a.warehouses * world
+    # ---- this rank's warehouse shard: weak scaling (a.warehouses per GPU) or strong (C4)
+    strong = a.total_warehouses is not None
+    W = a.total_warehouses if strong else a.warehouses * world
     lo, hi = chgen.warehouse_ranges(W, world)[rank]
     tables = chgen.generate(lo, hi, seed=1, mode=a.mode)
     hot = h.hot_path_tables(tables)
@@ -245,7 +406,9 @@ def main():
     n_c = len(tables["customer"]["c_id"])
     box = (key_box(tables["orders"], ("o_w_id", "o_d_id", "o_id")),
            key_box(tables["customer"], ("c_w_id", "c_d_id", "c_id")))
+    del tables
     pinned = {t: {c: torch.from_numpy(v).pin_memory() for c, v in cols.items()} for t, cols in hot.items()}
+    del hot
     h2d_bytes = sum(v.numel() * v.element_size() for cols in pinned.values() for v in cols.values())
     epoch = 1
     h.h2tap_load_snapshot(eng, pinned, epoch)
@@ -259,29 +422,33 @@ def main():
             dist.barrier()
         torch.cuda.synchronize()
 
+    def max_over_ranks(vals):
+        t = torch.tensor(vals, dtype=torch.float64, device="cuda")
+        if world > 1:
+            dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        return [float(x) for x in t.tolist()]
+
     plans = (("q6", h.H2TAP_Q6, Q6_P), ("q1", h.H2TAP_Q1, Q1_P), ("q18", h.H2TAP_Q18, Q18_P))
 
-    def step(flags):
-        # one batch on the resident snapshot: the three plans run back to back on the GPU and
-        # the library synchronises once (h2tap_run_queries)
-        rs = h.h2tap_run_queries(eng, [(plan, p, flags) for _, plan, p in plans])
+    def run_batch(sel, flags):
+        rs = h.h2tap_run_queries(eng, [(plan, p, flags) for name, plan, p in plans if name in sel])
         out = {}
-        for (name, _, _), r in zip(plans, rs):
+        for name, r in zip([n for n, _, _ in plans if n in sel], rs):
             out[name] = (r.device_ms, r.kernels if flags & h.H2TAP_QUERY_PROFILE else [], r.nrows,
-                         r.kernel_launches)
+                         r.kernel_launches, r.total_rows)
             if name == "q18":
                 dense_seen.append(r.plan_flags == 3)  # both join indexes perfect-hash
             h.h2tap_free(r)
         return out
 
     dense_seen = []
-
     dev_flags = h.H2TAP_RESULT_DEVICE
     prof_flags = h.H2TAP_RESULT_DEVICE | h.H2TAP_QUERY_PROFILE
+    ALL = ("q6", "q1", "q18")
     clocks = Clocks(local)  # sampled from warm-up to the end of the instrumented pass
     time.sleep(0.3)
     for _ in range(a.warmup):
-        step(dev_flags)
+        run_batch(ALL, dev_flags)
     barrier()
 
     def flush_l2():
@@ -295,39 +462,58 @@ def main():
     ends = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
     per_query = {"q6": [], "q1": [], "q18": []}
     launches = 0
-    n_pass = 0
+    n_pass = n_pass_total = 0
     barrier()
     for i in range(a.steps):
         flush_l2()
+        with torch.cuda.stream(stream):  # ~50 us sleep outside the events: the host enqueues the
+            torch.cuda._sleep(200_000)   # batch while the GPU sleeps (no launch gap inside)
         starts[i].record(stream)
-        out = step(dev_flags)
+        out = run_batch(ALL, dev_flags)
         ends[i].record(stream)
-        for q, (ms, ks, nrows, nl) in out.items():
+        for q, (ms, ks, nrows, nl, tot) in out.items():
             per_query[q].append(ms)
             launches += nl
-        n_pass = out["q18"][2]
+        n_pass, n_pass_total = out["q18"][2], out["q18"][4]
     barrier()
     step_ms_local = sum(s.elapsed_time(e) for s, e in zip(starts, ends)) / a.steps
+
+    # ---- the scans alone (not sharing a pass): Q6 by itself, Q1 by itself (C2 = Q1 at W=100).
+    # The query's own CUDA events (result.device_ms, recorded on the engine stream around its
+    # kernels); a ~50 us sleep kernel queued first lets the host enqueue the whole query before the
+    # GPU reaches it, so no launch latency lands inside the window
+    alone = {}
+    for q in ("q6", "q1"):
+        for _ in range(2):
+            run_batch((q,), dev_flags)
+        barrier()
+        ms = []
+        for _ in range(a.steps):
+            flush_l2()
+            with torch.cuda.stream(stream):
+                torch.cuda._sleep(200_000)
+            ms.append(run_batch((q,), dev_flags)[q][0])
+        alone[q] = float(np.median(ms))
+    barrier()
 
     # ---- instrumented pass (same K steps): per-kernel CUDA events for the roofline; a 30 us gate
     # kernel at each query start keeps host launch latency out of every kernel's event window
     kern = {}
     for i in range(a.steps):
         flush_l2()
-        out = step(prof_flags)
-        for q, (ms, ks, nrows, nl) in out.items():
+        out = run_batch(ALL, prof_flags)
+        for q, (ms, ks, nrows, nl, tot) in out.items():
             for kname, kms in ks:
                 kern.setdefault(kname, []).append(kms)
     barrier()
     clk = clocks.stop()
-    t = torch.tensor([step_ms_local], dtype=torch.float64, device="cuda")
-    if world > 1:
-        dist.all_reduce(t, op=dist.ReduceOp.MAX)
-    step_ms = float(t.item())
+    step_ms, q6_alone_ms, q1_alone_ms = max_over_ranks([step_ms_local, alone["q6"], alone["q1"]])
+    lat = {q: float(np.median(v)) for q, v in per_query.items()}
+    lat_max = dict(zip(lat, max_over_ranks(list(lat.values()))))
     nt = torch.tensor([n_ol], dtype=torch.float64, device="cuda")
-    if world > 1:  # weak scaling: every rank holds its own shard of W warehouses
+    if world > 1:
         dist.all_reduce(nt, op=dist.ReduceOp.SUM)
-    rows_total = 3 * int(nt.item())  # order_line rows all ranks scanned, x3 queries
+    rows_total = int(nt.item())  # order_line rows of all ranks, each counted once per step
     value = rows_total / (step_ms / 1e3)
 
     plan_dense = bool(dense_seen) and all(dense_seen)
@@ -337,6 +523,7 @@ def main():
                    else "v2" if os.environ.get("H2TAP_ORDER_CARRY") == "0" else "carry")
     dominant = max(kavg, key=kavg.get) if kavg else None
     peak, peak_src = peaks()
+    rpeak = read_stream_peak(h, eng, stream) if rank == 0 else None
     roof = None
     if dominant:
         b = alg_bytes(dominant, n_ol, n_o, n_c, n_pass, sort_passes, box if plan_dense else None)
@@ -347,6 +534,8 @@ def main():
                     "unit": "GB/s", "frac": round(ach / peak, 4), "traffic": tr,
                     "algorithmic_bytes_per_launch": int(b), "avg_launch_ms": round(kavg[dominant], 5),
                     "share_of_step": round(kavg[dominant] / step_ms_local, 4), "peak_source": peak_src,
+                    "read_stream_peak_gbs": rpeak,
+                    "frac_of_read_stream_peak": round(ach / rpeak, 4) if rpeak else None,
                     "timing": "CUDA events on the engine stream, instrumented pass of the same K steps"}
     kernels_summary = {}
     for k, v in kavg.items():
@@ -377,16 +566,14 @@ def main():
             h.h2tap_free(r)
     barrier()
     e2e_serial_s = (time.perf_counter() - t0) / e2e_steps
-    # pipelined: the same calls with H2TAP_LOAD_ASYNC | H2TAP_LOAD_BORROW (the pinned buffers are
-    # lent to the DMA and not modified), so step k's 1.2 GB upload (copy stream)
-    # overlaps step k-1's result read-back (D2H, the other PCIe direction) and the queries; each
-    # batch runs on the latest PUBLISHED epoch (k or k-1, reported per step) — double buffering
-    # (one rank only: with world > 1 the ranks could publish different epochs and a collective
-    # query must see one epoch everywhere)
+    # pipelined (reported separately): the same calls with H2TAP_LOAD_ASYNC | H2TAP_LOAD_BORROW, so
+    # step k's upload overlaps step k-1's result read-back and queries; each batch runs on the
+    # latest PUBLISHED epoch (lag reported) — one rank only (a collective batch must see one epoch
+    # on every rank)
     h.h2tap_sync(eng)
     barrier()
     lag = []
-    e2e_pipe_s = float("inf")
+    e2e_pipe_s = float("nan")
     if world == 1:
         for _ in range(3):  # warm-up: grows the device pool to the in-flight snapshot copies
             epoch += 1
@@ -405,54 +592,68 @@ def main():
         h.h2tap_sync(eng)  # the last upload is inside the timed region too
         e2e_pipe_s = (time.perf_counter() - t0) / e2e_steps
     barrier()
-    te = torch.tensor([e2e_serial_s, e2e_pipe_s], dtype=torch.float64, device="cuda")
-    if world > 1:
-        dist.all_reduce(te, op=dist.ReduceOp.MAX)
-    e2e_serial_s, e2e_pipe_s = (float(x) for x in te.tolist())
-    e2e_s = min(e2e_serial_s, e2e_pipe_s)
+    e2e_serial_s, = max_over_ranks([e2e_serial_s])
 
-    # ---- CPU oracle baseline (rank 0, N = 1 only, bounded sample)
-    cpu = None
+    # ---- CPU oracle baseline (rank 0, N = 1 only, bounded sample) and config C1
+    cpu = c1 = None
     if rank == 0 and world == 1 and not a.no_cpu_baseline:
         sample_w = 20
-        v, dt, n = cpu_oracle_sample(lo, sample_w, a.mode)
-        cpu = {"value": v, "unit": UNIT, "cores": 1, "kind": "oracle",
-               "sample": f"oracle Q6+Q1+Q18 once over W={sample_w} of the same warehouses "
-                         f"({n} order_line rows, {dt:.1f} s, single thread)"}
+        v, dt, n, core = cpu_oracle_sample(lo, sample_w, a.mode)
+        cpu = dict({"value": v, "unit": UNIT, "cores": 1, "kind": "oracle", "pinned_core": core,
+                    "sample": f"oracle Q6+Q1+Q18 once over W={sample_w} of the same warehouses "
+                              f"({n} order_line rows, {dt:.1f} s, single thread on core {core})"},
+                   **host_cpu())
+    if rank == 0 and world == 1 and not a.no_c1:
+        c1 = c1_line(h, a)
 
     if rank == 0:
         line = {
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": a.steps,
             "warmup": a.warmup, "ms_per_step": step_ms, "higher_is_better": True,
-            "scaling": "weak", "vs_baseline": None, "dtype": "int64", "data": "synthetic",
-            "config": {"workload": f"CH Q6+Q1+Q18 per step over W={a.warehouses} warehouses per GPU "
-                                   f"('{a.mode}' TPC-C population, seed 1)",
-                       "warehouses_per_gpu": a.warehouses, "order_line_rows_per_gpu": n_ol,
-                       "orders_rows_per_gpu": n_o, "customer_rows_per_gpu": n_c,
+            "scaling": "strong" if strong else "weak", "vs_baseline": None, "dtype": "int64",
+            "data": "synthetic",
+            "config": {"workload": (f"CH Q6+Q1+Q18 per step over W={W} warehouses split over {world} GPU(s)"
+                                    if strong else
+                                    f"CH Q6+Q1+Q18 per step over W={a.warehouses} warehouses per GPU")
+                                   + f" ('{a.mode}' TPC-C population, seed 1)",
+                       "warehouses_total": W, "warehouses_per_gpu": W / world,
+                       "order_line_rows_total": rows_total, "order_line_rows_rank0": n_ol,
+                       "orders_rows_rank0": n_o, "customer_rows_rank0": n_c,
+                       "rows_counted": ROWS_COUNTED,
                        "queries_per_step": 3, "parallelism": f"row-sharded by warehouse x{world}",
+                       "merge": ("peer-memory kernels over NVLink (Q6 allreduce, Q1 group lists, Q18 "
+                                 "range-partitioned ORDER BY; DESIGN.md §6)" if world > 1 else "none (1 GPU)"),
                        "scan_sharing": ("Q6 and Q1 of the batch share one pass over order_line "
-                                        "(latency_ms q6 includes it, q1 is its finalize; DESIGN.md "
-                                        "§4.5); every query computes its full result"
+                                        "(latency_ms.q6 includes it, q1 is its finalize; DESIGN.md "
+                                        "§4.5); every query computes its full result; the scans alone "
+                                        "are in latency_ms.q6_alone / q1_alone"
                                         if os.environ.get("H2TAP_SHARED_SCAN", "1") != "0" else "off"),
                        "l2": ("inputs > L2; between steps (outside events) 512 MB written then 256 MB read to flush L2"
                               if flush is not None else "inputs > L2 (no flush)")},
-            "latency_ms": {q: round(float(np.median(v)), 4) for q, v in per_query.items()},
-            "rows_per_s": {q: rows_total / 3 / (float(np.median(v)) / 1e3) for q, v in per_query.items()},
-            "q18_result_rows": n_pass,
+            "latency_ms": {"q6_q1_shared_scan_batch": round(lat_max["q6"] + lat_max["q1"], 4),
+                           "q6_in_batch": round(lat_max["q6"], 4), "q1_in_batch": round(lat_max["q1"], 4),
+                           "q18": round(lat_max["q18"], 4),
+                           "q6_alone": round(q6_alone_ms, 4), "q1_alone": round(q1_alone_ms, 4)},
+            "rows_per_s": {"q6_alone": rows_total / (q6_alone_ms / 1e3),
+                           "q1_alone": rows_total / (q1_alone_ms / 1e3),
+                           "q6_q1_batch": rows_total / ((lat_max["q6"] + lat_max["q1"]) / 1e3),
+                           "q18": rows_total / (lat_max["q18"] / 1e3)},
+            "q18_result_rows_total": n_pass_total, "q18_result_rows_rank0": n_pass,
             "roofline": roof,
             "kernels": kernels_summary,
             "cpu_baseline": cpu,
-            "e2e": {"value": rows_total / e2e_s, "unit": UNIT, "h2d_bytes_per_step": int(h2d_bytes),
-                    "d2h_bytes_per_step": int(d2h), "ms_per_step": e2e_s * 1e3, "steps": e2e_steps,
-                    "mode": "pipelined" if e2e_pipe_s <= e2e_serial_s else "serial",
-                    "serial_ms_per_step": e2e_serial_s * 1e3,
-                    "pipelined_ms_per_step": e2e_pipe_s * 1e3 if world == 1 else None,
-                    "pipelined_epoch_lag": sorted(set(lag)),
+            "c1": c1,
+            "e2e": {"value": rows_total / e2e_serial_s, "unit": UNIT, "h2d_bytes_per_step": int(h2d_bytes),
+                    "d2h_bytes_per_step": int(d2h), "ms_per_step": e2e_serial_s * 1e3, "steps": e2e_steps,
+                    "mode": "serial: each step's queries read that step's upload",
                     "how": "every step: full snapshot upload of the step's inputs from pinned host "
                            "buffers (h2tap_load_snapshot) + Q6/Q1/Q18 batch (h2tap_run_queries) + "
-                           "results copied to host; serial = load then queries; pipelined = "
-                           "H2TAP_LOAD_ASYNC|H2TAP_LOAD_BORROW, queries on the latest published "
-                           "epoch (lag in epochs listed)"},
+                           "results copied to host"},
+            "e2e_pipelined": ({"value": rows_total / e2e_pipe_s, "unit": UNIT, "ms_per_step": e2e_pipe_s * 1e3,
+                               "epoch_lag": sorted(set(lag)),
+                               "how": "H2TAP_LOAD_ASYNC|H2TAP_LOAD_BORROW: uploads overlap the previous "
+                                      "step's queries and read-back; each batch reads the latest "
+                                      "published epoch (lag in epochs listed)"} if world == 1 else None),
             "gpu_launches": int(launches),
             "clocks": clk,
         }
