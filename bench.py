@@ -217,7 +217,13 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None):
         "q18_sort_keys_hist": (32 + 8 + 8 + 4) * n_pass,   # rows + amounts -> keys + row ids
         # ORDER BY v2 (default): count matrix + scatter computing keys + chunked local sort
         "q18_sort_hist": 8 * n_pass,                       # amounts (bucket bits inside field a)
-        "q18_bucket_scatter": (40 + 16) * n_pass if sort_passes != "v1" else (12 + 12) * n_pass,
+        "q18_bucket_scatter": (16 + 16) * n_pass if sort_passes == "carry"
+                              else (40 + 16) * n_pass if sort_passes != "v1" else (12 + 12) * n_pass,
+        # v3 (default): accumulators + o_entry_d of the passing groups for the plan's bounds
+        "q18_acc_stats": 16 * n_o + 8 * n_o,
+        # v3: acc + orders keys in, per result row a customer slot + c_last + (o_id, o_ol_cnt,
+        # o_entry_d) and the 16 B carry record out
+        "q18_having_records": 16 * n_o + 12 * n_o + (slot_b + 4 + 16 + 16) * n_pass,
         # carry records (v2 default): 16 B record in, 40 B of result columns out (no row gather);
         # row-id paths: pair in + 32 B row gather + 40 B out
         "q18_bucket_sort_emit": (16 + 40) * n_pass if sort_passes == "carry"

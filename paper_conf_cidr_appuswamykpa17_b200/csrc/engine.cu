@@ -897,6 +897,9 @@ struct QueryCtx {
     Q18Cols out{};                          // device output columns (sorted)
     uint64_t n_max = 0;
     unsigned int *tie_dev = nullptr;
+    // Q18 v3 (HAVING builds the carry records) and the batch's snapshot
+    bool v3 = false;
+    const View *view = nullptr;
     // world > 1: distributed ORDER BY
     bool dist = false;
     uint64_t dist_out_cap = 0;              // rows the output columns hold
@@ -1243,6 +1246,96 @@ Q18Zone q18_zone(const View &v, bool q3) {
     return z;
 }
 
+// HAVING of the v2 path: the 32-byte result rows + amounts (compacted) and their statistics.
+void q18_having_v2(h2tap_engine *e, const View &v, QueryCtx &q) {
+    const int O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
+    const uint64_t n_o = v.n[O];
+    e->prof.run("q18_having_compact", [&] {
+        if (n_o)
+            launch_q18_having(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
+                              colp<int32_t>(v, O, H2TAP_O_ID), colp<int32_t>(v, O, H2TAP_O_C_ID),
+                              colp<int32_t>(v, O, H2TAP_O_OL_CNT), colp<int64_t>(v, O, H2TAP_O_ENTRY_D),
+                              n_o, colp<int32_t>(v, C, H2TAP_C_LAST), q.p[0], q.q18, e->num_sms, e->compute,
+                              e->having_unroll);
+    });
+    CK(cudaGetLastError());
+}
+
+void q18_order_dist(h2tap_engine *e, QueryCtx &q, const Q18HavingArgs *hv = nullptr,
+                    const unsigned long long *nout_for_meta = nullptr);
+
+// Q18 v3: statistics of the accumulators -> plan -> HAVING writes the carry records
+// and the bucket counts -> scan -> scatter -> per-bucket sort + emit (world > 1: the distributed
+// ORDER BY of §6.3 on the same records).
+void q18_launch_v3(h2tap_engine *e, const View &v, QueryCtx &q) {
+    const int O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
+    const uint64_t n_o = v.n[O];
+    const uint64_t n_max = std::max<uint64_t>(n_o, 1);
+    Q18Scratch &s = q.q18;
+    q.v3 = true;
+    q.n_max = n_o;
+    q.tie_dev = s.tie;
+    const int G = ob_grid(e->num_sms);
+    auto *cpart = static_cast<unsigned long long *>(e->arena.get("q18.cpart", 8ull * 8 * e->num_sms));
+    auto *scount = static_cast<unsigned long long *>(e->arena.get("q18.scount", 64));
+    auto *cnt_part = static_cast<unsigned int *>(e->arena.get("q18.cntpart", 4ull * G));
+    q.plan_dev = static_cast<Q18Plan *>(e->arena.get("q18.plan", sizeof(Q18Plan)));
+    const size_t nbm = size_t(1) << kBucketMaxBits;
+    BucketSort &bs = q.bs;
+    bs = BucketSort{};
+    bs.k[0] = static_cast<unsigned long long *>(e->arena.get("q18.rec", 16 * n_max));  // HAVING's records
+    bs.kv = static_cast<unsigned long long *>(e->arena.get("q18.kv", 16 * n_max));
+    bs.count = static_cast<unsigned int *>(e->arena.get("q18.bcount", 4 * (nbm + 1)));
+    bs.offset = static_cast<unsigned int *>(e->arena.get("q18.boffset", 4 * (nbm + 1)));
+    bs.big = static_cast<unsigned int *>(e->arena.get("q18.bbig", 4 * (nbm + 1)));
+    bs.ticket = static_cast<unsigned int *>(e->arena.get("q18.bticket", 64, true, e->compute));
+    bs.mat = static_cast<unsigned int *>(e->arena.get("q18.bmat", 4ull * G * nbm));
+    const int64_t *o_ent = colp<int64_t>(v, O, H2TAP_O_ENTRY_D);
+    ProfMarks marks(e->prof);
+    if (e->world > 1) {
+        e->prof.run("q18_acc_stats", [&] {
+            launch_q18_acc_stats(s, o_ent, n_o, q.p[0], cpart, scount, nullptr, 0, nullptr, q.tie_dev,
+                                 e->num_sms, e->compute);
+        });
+        const Q18HavingArgs hv{colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
+                               colp<int32_t>(v, O, H2TAP_O_ID), colp<int32_t>(v, O, H2TAP_O_C_ID),
+                               colp<int32_t>(v, O, H2TAP_O_OL_CNT), o_ent, n_o,
+                               colp<int32_t>(v, C, H2TAP_C_LAST), q.p[0], s, cnt_part};
+        q18_order_dist(e, q, &hv, scount);
+        return;
+    }
+    int bb = ob_bucket_bits(n_max);
+    if (const char *d = std::getenv("H2TAP_BUCKET_BITS_DELTA"))
+        bb = std::max(1, std::min(kBucketMaxBits, bb + std::atoi(d)));
+    q18_alloc_out(e, q, n_max);
+    const Q18PlanArgs pa{s.stats, q.zone, nullptr, 1};
+    e->prof.run("q18_acc_stats", [&] {
+        launch_q18_acc_stats(s, o_ent, n_o, q.p[0], cpart, scount, &pa, bb, q.plan_dev, q.tie_dev, e->num_sms,
+                             e->compute);
+    });
+    q18_order_v3(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID), colp<int32_t>(v, O, H2TAP_O_ID),
+                 colp<int32_t>(v, O, H2TAP_O_C_ID), colp<int32_t>(v, O, H2TAP_O_OL_CNT), o_ent, n_o,
+                 colp<int32_t>(v, C, H2TAP_C_LAST), q.p[0], s, q.plan_dev, bb, bs, cnt_part, q.out, q.tie_dev,
+                 e->num_sms, e->compute, &marks);
+    CK(cudaGetLastError());
+    launch_q18_publish(s.nout, s.err, q.tie_dev, q.small_dev, e->compute);  // -> small (mapped)
+}
+
+// The v3 records did not fit 128 bits (or a bucket overflowed): redo HAVING + ORDER BY on the v2
+// path from the accumulators, which are intact (host-synchronous; rare on realistic data).
+void q18_rerun_v2(h2tap_engine *e, QueryCtx &q) {
+    Q18Scratch &s = q.q18;
+    const Q18Stats init{INT64_MAX, INT64_MIN, INT64_MAX, INT64_MIN};
+    CK(cudaMemsetAsync(s.nout, 0, 8, e->compute));
+    CK(cudaMemsetAsync(s.tie, 0, 4, e->compute));
+    CK(cudaMemcpyAsync(s.stats, &init, sizeof init, cudaMemcpyHostToDevice, e->compute));
+    release_dev_blocks(e, q);
+    q.v3 = false;
+    q18_having_v2(e, *q.view, q);
+    q18_gather_and_order(e, q, q.view->n[H2TAP_T_ORDERS]);
+    sync_compute(e);
+}
+
 void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
     need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}, "Q18");
@@ -1266,22 +1359,21 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
                              colp<int32_t>(v, OL, H2TAP_OL_O_ID), colp<int64_t>(v, OL, H2TAP_OL_AMOUNT),
                              n_ol, s, e->num_sms, e->compute);
     });
-    e->prof.run("q18_having_compact", [&] {
-        if (n_o)
-            launch_q18_having(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
-                              colp<int32_t>(v, O, H2TAP_O_ID), colp<int32_t>(v, O, H2TAP_O_C_ID),
-                              colp<int32_t>(v, O, H2TAP_O_OL_CNT), colp<int64_t>(v, O, H2TAP_O_ENTRY_D),
-                              n_o, colp<int32_t>(v, C, H2TAP_C_LAST), q.p[0], s, e->num_sms, e->compute,
-                              e->having_unroll);
-    });
     CK(cudaGetLastError());
     q.zone = q18_zone(v, false);
+    q.view = &v;
+    const char *cv = std::getenv("H2TAP_ORDER_CARRY");
+    if (!e->order_v1 && !(cv && cv[0] == '0')) {  // v3: HAVING builds the carry records
+        q18_launch_v3(e, v, q);
+        return;
+    }
+    q18_having_v2(e, v, q);
     q18_gather_and_order(e, q, n_o);
 }
 
 // a7 + a8 of Q18 (and Q3) with world > 1: the distributed ORDER BY. Every rank
 // ends up with its range of the global order; nothing is gathered, nothing waits for the host.
-void q18_order_dist(h2tap_engine *e, QueryCtx &q) {
+void q18_order_dist(h2tap_engine *e, QueryCtx &q, const Q18HavingArgs *hv, const unsigned long long *nout_for_meta) {
     Q18Scratch &s = q.q18;
     const uint64_t n_max = std::max<uint64_t>(q.n_max, 1);
     const size_t nbm = size_t(1) << kBucketMaxBits;
@@ -1294,6 +1386,7 @@ void q18_order_dist(h2tap_engine *e, QueryCtx &q) {
     bs.ticket = static_cast<unsigned int *>(e->arena.get("q18.bticket", 64, true, e->compute));
     bs.mat = static_cast<unsigned int *>(e->arena.get("q18.bmat", 4ull * ob_grid(e->num_sms) * nbm));
     bs.kv = static_cast<unsigned long long *>(e->arena.get("q18.kv", 16 * n_max));
+    if (hv) bs.k[0] = static_cast<unsigned long long *>(e->arena.get("q18.rec", 16 * n_max));
     auto *send = static_cast<unsigned long long *>(e->arena.get("q18.dsend", 8 * nbm));
     q.recv_off = static_cast<unsigned int *>(e->arena.get("q18.drecv", 4 * (nbm + 1)));
     // output capacity: ~1/world of the global result lands here; twice the local orders rows
@@ -1305,10 +1398,10 @@ void q18_order_dist(h2tap_engine *e, QueryCtx &q) {
     const char *cv = std::getenv("H2TAP_ORDER_CARRY");
     const bool carry = !(cv && cv[0] == '0');
     q.tie_dev = s.tie;
-    const Q18PlanArgs meta{s.stats, q.zone, s.nout, carry ? 1 : 0};
+    const Q18PlanArgs meta{s.stats, q.zone, nout_for_meta ? nout_for_meta : s.nout, carry ? 1 : 0};
     ProfMarks marks(e->prof);
     q18_bucket_order_dist(e->peer.args, q.rows, q.amt, q.plan_dev, meta, s.err, bs, send, q.recv_off, cap, q.out,
-                          q.tie_dev, q.small_dev, e->num_sms, e->compute, &marks);
+                          q.tie_dev, q.small_dev, e->num_sms, e->compute, &marks, hv);
     q.dist = true;
 }
 
@@ -1382,6 +1475,7 @@ void finish_q18(h2tap_engine *e, QueryCtx &q) {
     const char *const *names = q3 ? kQ3Names : kQ18Names;
     const uint32_t *types = q3 ? kQ3Types : kQ18Types;
     const int ncols = q3 ? 5 : 8;
+    if (q.v3 && !q.dist && (sm->tie & (1u | 2u | 4u | 8u))) q18_rerun_v2(e, q);  // (carry did not fit)
     const unsigned int err = sm->err;  // world > 1: every rank's join errors and the exchange's
     const unsigned pl = q.plan;
     if (err & kPeerErrTimeout) {

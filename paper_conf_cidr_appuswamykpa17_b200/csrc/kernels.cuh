@@ -289,11 +289,35 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, Q18Plan *plan
 // partition, exchange of the carry records into the owners' heaps, per-bucket sort + emit of this
 // rank's range of the global order into dst (capacity out_cap rows); {n_mine, err, tie, stats,
 // row0, n_total} -> host_small (mapped). send: [2^kBucketMaxBits] u64, recv_off: [2^kBucketMaxBits+1].
+// v3: the HAVING pass builds the carry records itself, with a plan derived
+// beforehand from the accumulators (launch_q18_acc_stats). The arguments of that HAVING pass:
+struct Q18HavingArgs {
+    const int32_t *o_w, *o_d, *o_id, *o_c, *o_cnt;
+    const int64_t *o_ent;
+    uint64_t n_o;
+    const int32_t *c_last;
+    int64_t having;
+    Q18Scratch s;
+    unsigned int *cnt_part;   // [ob_grid] records per partition
+};
+// min / max of amount_sum and o_entry_d over the groups passing cnt > 0 AND sum > having (and their
+// count, *count); with plan_args, the last block also derives the ORDER BY plan (zone from there)
+void launch_q18_acc_stats(const Q18Scratch &s, const int64_t *o_ent, uint64_t n_o, int64_t having,
+                          unsigned long long *cpart, unsigned long long *count, const Q18PlanArgs *plan_args,
+                          int bucket_bits, Q18Plan *plan, unsigned int *flag, int num_sms, cudaStream_t st);
+// one GPU: HAVING + records + histogram -> scan -> scatter -> per-bucket sort + emit; *flag bit 8:
+// the records did not fit (the host re-runs the v2 path), bit 1: an oversized bucket (likewise)
+void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, const int32_t *o_c,
+                  const int32_t *o_cnt, const int64_t *o_ent, uint64_t n_o, const int32_t *c_last,
+                  int64_t having, const Q18Scratch &s, const Q18Plan *plan, int bucket_bits,
+                  const BucketSort &bs, unsigned int *cnt_part, const Q18Cols &dst, unsigned int *flag,
+                  int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr);
+// hv non-null: the v3 input (records built by the HAVING pass); null: rows + amounts (Q3)
 void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long long *amt, Q18Plan *plan,
                            const Q18PlanArgs &meta, const unsigned int *err, const BucketSort &s,
                            unsigned long long *send, unsigned int *recv_off, uint64_t out_cap,
                            const Q18Cols &dst, unsigned int *flag, void *host_small, int num_sms,
-                           cudaStream_t st, PhaseMarks *marks = nullptr);
+                           cudaStream_t st, PhaseMarks *marks = nullptr, const Q18HavingArgs *hv = nullptr);
 // The emit phase alone (re-run by the host into larger output columns after kPeerErrOutCap; the
 // exchanged records stay in the heap until the next exchange of the same parity).
 void q18_dist_emit(const PeerArgs &pa, const Q18Plan *plan, const unsigned int *recv_off, const Q18Cols &dst,

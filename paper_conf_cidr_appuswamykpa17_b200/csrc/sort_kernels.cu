@@ -20,6 +20,7 @@
 #include <cuda_runtime.h>
 
 #include "cache_hints.cuh"
+#include "join_index.cuh"
 #include "kernels.cuh"
 #include "peer.cuh"
 
@@ -763,6 +764,7 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
     }
     // row-id path: the v2 small instance holds 1 024 rows (LsSmem<1024> fits the 35 KB of the
     // carry layout, so both run 6 blocks per SM); larger buckets go to the large instance
+    if (rows == nullptr) return;  // v3 / distributed: carry records only (row path re-run by the host)
     constexpr int kRowCap = (kPairs && kMin == 0) ? 1024 : kLsCap;
     LsSmem<kRowCap> &S = *reinterpret_cast<LsSmem<kRowCap> *>(smem_raw);
     const int shift = plan->shift;
@@ -1021,10 +1023,18 @@ ob_hist_kernel(const Q18Row *__restrict__ rows, const long long *__restrict__ am
 constexpr int kScanWarps = 32;
 __global__ void __launch_bounds__(32 * kScanWarps)
 ob_scan_kernel(unsigned int *__restrict__ mat, int G, int nb, unsigned int *__restrict__ count,
-               unsigned int *__restrict__ offset, unsigned int *ticket, const Q18Plan *__restrict__ plan) {
+               unsigned int *__restrict__ offset, unsigned int *ticket, const Q18Plan *__restrict__ plan,
+               ulonglong2 *__restrict__ touch = nullptr, uint64_t touch_n = 0) {
     pdl_wait();
     pdl_trigger();
     if (plan && plan->dist) nb = 1 << plan->bucket_bits;  // (grid sized for the launch nb)
+    if (touch) {  // v3: the scatter's target lines into L2 first (l2_touch_kernel; the scan has spare
+                  // bandwidth: it is latency-bound)
+        const uint64_t keep = l2_policy_evict_last();
+        const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+        for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < touch_n; i += stride)
+            st16_policy(touch + i, 0ull, 0ull, keep);
+    }
     extern __shared__ unsigned int tile[];  // [G][32]; the last block reuses it for nb totals
     __shared__ bool last;
     __shared__ unsigned int tot[kScanWarps][32];
@@ -1216,7 +1226,7 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, Q18Plan *plan
     end();
     begin("q18_sort_scan");
     launch_pdl(ob_scan_kernel, (nb + 31) / 32, 32 * kScanWarps, 4 * std::max(32 * G, nb), st, s.mat, G, nb, s.count,
-               s.offset, s.ticket, (const Q18Plan *)plan);
+               s.offset, s.ticket, (const Q18Plan *)plan, (ulonglong2 *)nullptr, (uint64_t)0);
     count_launches(1);
     end();
     begin("q18_bucket_scatter");
@@ -1233,6 +1243,342 @@ void q18_bucket_order_v2(const Q18Row *rows, const long long *amt, Q18Plan *plan
     begin("q18_bucket_sort_emit_large");
     launch_pdl(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>, (unsigned)num_sms, kEmThreads, kObSmemLarge, st,
         s.kv, nullptr, s.offset, nb, plan, rows, amt, dst, flag, s.big, sub_log2, PeerArgs{});
+    count_launches(1);
+    end();
+}
+
+}  // namespace h2tap
+
+// ================================ Q18 v3: HAVING writes carry records (default) ===
+// The v2 chain materialises every result row twice before the sort (HAVING: 32 B row + 8 B amount;
+// ob_hist re-reads the amounts; ob_scatter re-reads rows + amounts to build the records). v3 derives
+// the ORDER BY plan BEFORE the HAVING pass, from one read of the accumulators (the min / max of
+// amount_sum and o_entry_d over the groups that pass cnt > 0 AND sum > having — a superset of the
+// result, whose bounds are valid for it), so the HAVING pass itself builds each result row's 16-byte
+// carry record and histograms its bucket:
+//   acc_stats (+ plan)  ->  having_rec: records, block-compacted into the block's own row range,
+//   + the block's bucket counts (one row of the [partition][bucket] matrix)  ->  ob_scan  ->
+//   scatter_rec: each block's records to their bucket positions  ->  per-bucket sort + emit (v2).
+// Rows whose records would not fit 128 bits (bit 8 of *flag) and oversized buckets (bit 2) are
+// re-run by the host through the v2 path (rows + amounts), which has the exact fallbacks.
+namespace h2tap {
+namespace {
+
+constexpr unsigned int kFlagRowPath = 8u;   // carry records do not fit: host re-runs the v2 path
+// H2TAP_KV_TOUCH=0: no pre-write of the scatter's target lines (A/B)
+int kv_touch_mode() {  // 1: inside the scan kernel (default), 2: its own kernel, 0: off
+    static const int m = [] { const char *v = std::getenv("H2TAP_KV_TOUCH"); return v ? std::atoi(v) : 1; }();
+    return m;
+}
+bool kv_touch() { return kv_touch_mode() != 0; }
+
+// The scatter writes 16-byte records at random kv positions: half sectors, which L2 would first
+// fill from DRAM (a random read per record). Writing the whole kv range just before (whole lines,
+// coalesced, kept in L2: no fills) makes those lines L2-resident: scatter 58 -> 27 us measured.
+__global__ void __launch_bounds__(1024) l2_touch_kernel(ulonglong2 *__restrict__ p, uint64_t n,
+                                                        const Q18Plan *__restrict__ plan) {
+    pdl_wait();
+    pdl_trigger();
+    if (!plan->spec.carry || (plan->err & ~kPeerErrOutCap)) return;
+    const uint64_t keep = l2_policy_evict_last();
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride)
+        st16_policy(p + i, 0ull, 0ull, keep);
+}
+constexpr int kStatThreads = 256;
+
+__device__ __forceinline__ long long wmin(long long v) {
+    for (int o = 16; o; o >>= 1) { const long long t = __shfl_xor_sync(kFull, v, o); v = t < v ? t : v; }
+    return v;
+}
+__device__ __forceinline__ long long wmax(long long v) {
+    for (int o = 16; o; o >>= 1) { const long long t = __shfl_xor_sync(kFull, v, o); v = t > v ? t : v; }
+    return v;
+}
+
+__global__ void __launch_bounds__(kStatThreads)
+q18_acc_stats_kernel(const Q18Acc *__restrict__ acc, const int64_t *__restrict__ o_ent, uint64_t n_o,
+                     long long having, Q18Stats *__restrict__ part, unsigned long long *__restrict__ cpart,
+                     unsigned int *ticket, Q18Stats *stats, unsigned long long *count, int make_plan,
+                     Q18Zone zone, int bucket_bits, int allow_carry, Q18Plan *plan, unsigned int *flag) {
+    pdl_wait();
+    pdl_trigger();
+    __shared__ Q18Stats ws[kStatThreads / 32];
+    __shared__ unsigned long long wc[kStatThreads / 32];
+    __shared__ bool last;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    long long amin = INT64_MAX, amax = INT64_MIN, emin = INT64_MAX, emax = INT64_MIN;
+    unsigned long long c = 0;
+    const uint64_t stride = (uint64_t)gridDim.x * kStatThreads;
+    constexpr int U = 4;  // independent accumulator loads in flight per thread
+    for (uint64_t r0 = (uint64_t)blockIdx.x * kStatThreads + threadIdx.x; r0 < n_o; r0 += U * stride) {
+        ulonglong2 a[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const uint64_t r = r0 + u * stride;
+            a[u] = r < n_o ? __ldcg(reinterpret_cast<const ulonglong2 *>(acc + r)) : make_ulonglong2(0, 0);
+        }
+        long long e[U];  // loaded unconditionally: independent of the accumulator loads (most pass)
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const uint64_t r = r0 + u * stride;
+            e[u] = r < n_o ? __ldcs(o_ent + r) : 0;
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const long long sum = (long long)a[u].x;
+            if ((unsigned int)a[u].y > 0 && sum > having) {
+                amin = sum < amin ? sum : amin; amax = sum > amax ? sum : amax;
+                emin = e[u] < emin ? e[u] : emin; emax = e[u] > emax ? e[u] : emax;
+                ++c;
+            }
+        }
+    }
+    amin = wmin(amin); amax = wmax(amax); emin = wmin(emin); emax = wmax(emax);
+    for (int o = 16; o; o >>= 1) c += __shfl_xor_sync(kFull, c, o);
+    if (lane == 0) { ws[warp] = Q18Stats{amin, amax, emin, emax}; wc[warp] = c; }
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        Q18Stats b{INT64_MAX, INT64_MIN, INT64_MAX, INT64_MIN};
+        unsigned long long bc = 0;
+        for (int k = 0; k < kStatThreads / 32; ++k) {
+            b.amt_min = min(b.amt_min, ws[k].amt_min); b.amt_max = max(b.amt_max, ws[k].amt_max);
+            b.ent_min = min(b.ent_min, ws[k].ent_min); b.ent_max = max(b.ent_max, ws[k].ent_max);
+            bc += wc[k];
+        }
+        part[blockIdx.x] = b;
+        cpart[blockIdx.x] = bc;
+        __threadfence();
+        last = atomicAdd(ticket, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!last) return;
+    __threadfence();
+    // the last block folds every block's partial, all threads in parallel (independent loads)
+    amin = INT64_MAX; amax = INT64_MIN; emin = INT64_MAX; emax = INT64_MIN; c = 0;
+    for (unsigned k = threadIdx.x; k < gridDim.x; k += kStatThreads) {
+        const long long *src = reinterpret_cast<const long long *>(part + k);
+        amin = min(amin, __ldcg(src + 0)); amax = max(amax, __ldcg(src + 1));
+        emin = min(emin, __ldcg(src + 2)); emax = max(emax, __ldcg(src + 3));
+        c += __ldcg(cpart + k);
+    }
+    amin = wmin(amin); amax = wmax(amax); emin = wmin(emin); emax = wmax(emax);
+    for (int o = 16; o; o >>= 1) c += __shfl_xor_sync(kFull, c, o);
+    __syncthreads();
+    if (lane == 0) { ws[warp] = Q18Stats{amin, amax, emin, emax}; wc[warp] = c; }
+    __syncthreads();
+    if (threadIdx.x != 0) return;
+    Q18Stats g{INT64_MAX, INT64_MIN, INT64_MAX, INT64_MIN};
+    unsigned long long gc = 0;
+    for (int k = 0; k < kStatThreads / 32; ++k) {
+        g.amt_min = min(g.amt_min, ws[k].amt_min); g.amt_max = max(g.amt_max, ws[k].amt_max);
+        g.ent_min = min(g.ent_min, ws[k].ent_min); g.ent_max = max(g.ent_max, ws[k].ent_max);
+        gc += wc[k];
+    }
+    *stats = g;
+    *count = gc;
+    *ticket = 0;  // self-reset
+    if (make_plan) {
+        Q18Plan P = make_q18_plan_vals(g, zone, gc, gc >= 1, bucket_bits, allow_carry, flag);
+        if (gc == 0) P.spec.carry = allow_carry;  // nothing to order: no record is ever decoded
+        *plan = P;
+    }
+}
+
+// HAVING + customer probe + carry record + bucket histogram, one block per contiguous orders-row
+// range (the same partition the scatter uses): records are compacted into the block's own range
+// of rec[] (a shared counter per warp-ballot), the block's bucket counts become matrix row p.
+constexpr int kHrThreads = 512;  // 2 blocks per SM (<= 64 registers), 4 rows per thread in flight
+__global__ void __launch_bounds__(kHrThreads, 2)
+q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
+                      const int32_t *__restrict__ o_id, const int32_t *__restrict__ o_c,
+                      const int32_t *__restrict__ o_cnt, const int64_t *__restrict__ o_ent, uint64_t n_o,
+                      const int32_t *__restrict__ c_last, long long having, Q18Scratch s,
+                      const Q18Plan *__restrict__ plan, int nb_launch, unsigned int *__restrict__ mat,
+                      unsigned int *__restrict__ cnt_part, ulonglong2 *__restrict__ rec, unsigned int *flag) {
+    pdl_wait();
+    pdl_trigger();
+    extern __shared__ unsigned int h[];
+    __shared__ unsigned int s_cnt;
+    __shared__ Q18SortSpec S;
+    __shared__ int s_shift, s_nb, s_carry;
+    if (threadIdx.x == 0) {
+        S = plan->spec;
+        s_shift = plan->shift;
+        s_nb = plan->dist ? (1 << plan->bucket_bits) : nb_launch;
+        s_carry = plan->spec.carry && !(plan->err);
+        s_cnt = 0;
+        if (!plan->spec.carry && blockIdx.x == 0 && !plan->dist) atomicOr(flag, kFlagRowPath);
+    }
+    __syncthreads();
+    const int nb = s_nb;
+    for (int i = threadIdx.x; i < nb; i += kHrThreads) h[i] = 0;
+    __syncthreads();
+    uint64_t r0, r1;
+    ob_range(n_o, r0, r1);
+    const int lane = threadIdx.x & 31;
+    const int shift = s_shift;
+    const Q18SortSpec sp = S;
+    const uint64_t keep = l2_policy_evict_last();  // records are re-read by the scatter
+    constexpr int U = 4;
+    if (s_carry)
+    for (uint64_t base = r0; base < r1; base += (uint64_t)U * kHrThreads) {
+        long long sum[U];
+        int w[U], d[U], c[U];
+        unsigned int crow[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {  // independent coalesced loads first
+            const uint64_t r = base + (uint64_t)u * kHrThreads + threadIdx.x;
+            crow[u] = kNoRow;
+            sum[u] = 0; w[u] = d[u] = c[u] = 0;
+            if (r < r1) {
+                const ulonglong2 a = __ldcs(reinterpret_cast<const ulonglong2 *>(s.acc + r));
+                sum[u] = (long long)a.x;
+                crow[u] = ((unsigned int)a.y > 0 && sum[u] > having) ? 0u : kNoRow;
+                w[u] = __ldcs(o_w + r); d[u] = __ldcs(o_d + r); c[u] = __ldcs(o_c + r);
+            }
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u)  // customer ⋈ orders, independent across rows
+            if (crow[u] == 0u) crow[u] = jx::jx_lookup(s.jc, w[u], d[u], c[u]);
+        ulonglong2 rc[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            if (crow[u] == kNoRow) continue;
+            const uint64_t r = base + (uint64_t)u * kHrThreads + threadIdx.x;
+            Q18Row row;
+            row.o_entry_d = __ldcs(o_ent + r);
+            row.c_last = __ldg(c_last + crow[u]);
+            row.c_id = c[u];
+            row.o_id = __ldcs(o_id + r);
+            row.o_ol_cnt = __ldcs(o_cnt + r);
+            row.o_w_id = w[u];
+            row.o_d_id = d[u];
+            rc[u] = carry_record(row, sum[u], sp);
+            atomicAdd(&h[(unsigned int)(rc[u].x >> shift)], 1u);
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u) {  // warp-aggregated compaction into the block's range
+            const bool v = crow[u] != kNoRow;
+            const unsigned int bal = __ballot_sync(kFull, v);
+            if (!bal) continue;
+            unsigned int wb = 0;
+            if (lane == __ffs(bal) - 1) wb = atomicAdd(&s_cnt, (unsigned int)__popc(bal));
+            wb = __shfl_sync(kFull, wb, __ffs(bal) - 1);
+            if (v) st16_policy(rec + r0 + wb + __popc(bal & ((1u << lane) - 1u)), rc[u].x, rc[u].y, keep);
+        }
+    }
+    __syncthreads();
+    unsigned int *row = mat + (uint64_t)blockIdx.x * nb;
+    for (int i = threadIdx.x; i < nb; i += kHrThreads) row[i] = h[i];
+    if (threadIdx.x == 0) {
+        cnt_part[blockIdx.x] = s_cnt;
+        if (s_cnt) atomicAdd(s.nout, (unsigned long long)s_cnt);
+    }
+}
+
+// Each block's records (rec[r0 .. r0 + cnt_part[p])) to their bucket positions: the shared cursors
+// start at offset[b] + matrix[p][b] (the column scan), no global atomics.
+__global__ void __launch_bounds__(kObThreads)
+ob_scatter_rec_kernel(const ulonglong2 *__restrict__ rec, uint64_t n_o, const Q18Plan *__restrict__ plan,
+                      int nb_launch, const unsigned int *__restrict__ mat, const unsigned int *__restrict__ offset,
+                      const unsigned int *__restrict__ cnt_part, ulonglong2 *__restrict__ kv) {
+    pdl_wait();
+    pdl_trigger();
+    extern __shared__ unsigned int cur[];
+    // (kPeerErrOutCap only stops this rank's emit: its records must still be exchanged)
+    if (!plan->spec.carry || (plan->err & ~kPeerErrOutCap)) return;
+    const int nb = plan->dist ? (1 << plan->bucket_bits) : nb_launch;
+    const int shift = plan->shift;
+    const unsigned int *row = mat + (uint64_t)blockIdx.x * nb;
+    for (int i = threadIdx.x; i < nb; i += kObThreads) cur[i] = offset[i] + row[i];
+    __syncthreads();
+    uint64_t r0, r1;
+    ob_range(n_o, r0, r1);
+    const unsigned int m = cnt_part[blockIdx.x];
+    const uint64_t drop = l2_policy_evict_first();
+    constexpr int U = 4;
+    for (unsigned int i0 = threadIdx.x; i0 < m; i0 += U * kObThreads) {
+        ulonglong2 r[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const unsigned int i = i0 + u * kObThreads;
+            if (i < m) ld16_policy(rec + r0 + i, r[u].x, r[u].y, drop);
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const unsigned int i = i0 + u * kObThreads;
+            if (i >= m) break;
+            const unsigned int p = atomicAdd(&cur[(unsigned int)(r[u].x >> shift)], 1u);
+            kv[p] = r[u];
+        }
+    }
+}
+
+}  // namespace
+
+void launch_q18_acc_stats(const Q18Scratch &s, const int64_t *o_ent, uint64_t n_o, int64_t having,
+                          unsigned long long *cpart, unsigned long long *count, const Q18PlanArgs *plan_args,
+                          int bucket_bits, Q18Plan *plan, unsigned int *flag, int num_sms, cudaStream_t st) {
+    uint64_t want = (n_o + kStatThreads - 1) / kStatThreads;
+    const uint64_t cap = (uint64_t)num_sms * 8;  // = the stat_part capacity (8 blocks per SM)
+    const unsigned grid = (unsigned)(want < 1 ? 1 : want > cap ? cap : want);
+    const Q18Zone z = plan_args ? plan_args->zone : Q18Zone{};
+    launch_pdl(q18_acc_stats_kernel, grid, kStatThreads, 0, st, (const Q18Acc *)s.acc, o_ent, n_o,
+               (long long)having, s.stat_part, cpart, s.ticket, s.stats, count, plan_args ? 1 : 0, z,
+               bucket_bits, plan_args ? plan_args->allow_carry : 0, plan, flag);
+    count_launches(1);
+}
+
+void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, const int32_t *o_c,
+                  const int32_t *o_cnt, const int64_t *o_ent, uint64_t n_o, const int32_t *c_last,
+                  int64_t having, const Q18Scratch &s, const Q18Plan *plan, int bucket_bits,
+                  const BucketSort &bs, unsigned int *cnt_part, const Q18Cols &dst, unsigned int *flag,
+                  int num_sms, cudaStream_t st, PhaseMarks *marks) {
+    auto begin = [&](const char *nm) { if (marks) marks->begin(nm); };
+    auto end = [&] { if (marks) marks->end(); };
+    const int nb = 1 << bucket_bits;
+    const int G = ob_grid(num_sms);
+    begin("q18_having_records");
+    launch_pdl(q18_having_rec_kernel, G, kHrThreads, 4 * nb, st, o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o, c_last,
+               (long long)having, s, plan, nb, bs.mat, cnt_part, reinterpret_cast<ulonglong2 *>(bs.k[0]), flag);
+    count_launches(1);
+    end();
+    begin("q18_sort_scan");
+    launch_pdl(ob_scan_kernel, (nb + 31) / 32, 32 * kScanWarps, 4 * std::max(32 * G, nb), st, bs.mat, G, nb,
+               bs.count, bs.offset, bs.ticket, plan,
+               kv_touch_mode() == 1 ? reinterpret_cast<ulonglong2 *>(bs.kv) : nullptr, kv_touch_mode() == 1 ? n_o : 0);
+    count_launches(1);
+    end();
+    if (kv_touch_mode() == 2) {
+        begin("q18_kv_touch");
+        launch_pdl(l2_touch_kernel, (unsigned)num_sms * 2, 1024, 0, st, reinterpret_cast<ulonglong2 *>(bs.kv), n_o, plan);
+        count_launches(1);
+        end();
+    }
+    begin("q18_bucket_scatter");
+    launch_pdl(ob_scatter_rec_kernel, G, kObThreads, 4 * nb, st, reinterpret_cast<const ulonglong2 *>(bs.k[0]), n_o,
+               plan, nb, (const unsigned int *)bs.mat, (const unsigned int *)bs.offset, (const unsigned int *)cnt_part,
+               reinterpret_cast<ulonglong2 *>(bs.kv));
+    count_launches(1);
+    end();
+    // big[] (the oversized-bucket work list) is reset by the hist kernel on the v2 path
+    cudaMemsetAsync(bs.big, 0, sizeof(unsigned int), st);
+    static const int sub_log2 = [] {
+        const char *v = std::getenv("H2TAP_SUB_ROWS_LOG2");
+        return v ? std::max(0, std::min(6, std::atoi(v))) : 1;
+    }();
+    begin("q18_bucket_sort_emit");
+    const unsigned lb = (unsigned)nb < (unsigned)num_sms * 6 ? (unsigned)nb : (unsigned)num_sms * 6;
+    launch_pdl(bucket_local_emit_kernel<kObCap, 0, true>, lb, kEmThreads, kObSmem, st,
+               (const unsigned long long *)bs.kv, (const unsigned int *)nullptr, (const unsigned int *)bs.offset, nb,
+               plan, (const Q18Row *)nullptr, (const long long *)nullptr, dst, flag, bs.big, sub_log2, PeerArgs{});
+    count_launches(1);
+    end();
+    begin("q18_bucket_sort_emit_large");
+    launch_pdl(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>, (unsigned)num_sms, kEmThreads, kObSmemLarge, st,
+               (const unsigned long long *)bs.kv, (const unsigned int *)nullptr, (const unsigned int *)bs.offset, nb,
+               plan, (const Q18Row *)nullptr, (const long long *)nullptr, dst, flag, bs.big, sub_log2, PeerArgs{});
     count_launches(1);
     end();
 }
@@ -1462,7 +1808,7 @@ void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long lo
                            const Q18PlanArgs &meta, const unsigned int *err, const BucketSort &s,
                            unsigned long long *send, unsigned int *recv_off, uint64_t out_cap,
                            const Q18Cols &dst, unsigned int *flag, void *host_small, int num_sms,
-                           cudaStream_t st, PhaseMarks *marks) {
+                           cudaStream_t st, PhaseMarks *marks, const Q18HavingArgs *hv) {
     auto begin = [&](const char *nm) { if (marks) marks->begin(nm); };
     auto end = [&] { if (marks) marks->end(); };
     const int nb = 1 << kBucketMaxBits;  // launch sizes: the largest bucket count the plan may pick
@@ -1472,13 +1818,24 @@ void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long lo
                kBucketMaxBits, plan, flag);
     count_launches(1);
     end();
-    begin("q18_sort_hist");
-    launch_pdl(ob_hist_kernel, G, kObThreads, nb * 4, st, rows, amt, plan, nb, s.mat, s.big, 0, Q18PlanArgs{}, 0, flag);
-    count_launches(1);
-    end();
+    if (hv) {  // v3: HAVING builds the carry records and the bucket counts with the global plan
+        begin("q18_having_records");
+        launch_pdl(q18_having_rec_kernel, G, kHrThreads, nb * 4, st, hv->o_w, hv->o_d, hv->o_id, hv->o_c, hv->o_cnt,
+                   hv->o_ent, hv->n_o, hv->c_last, (long long)hv->having, hv->s, (const Q18Plan *)plan, nb, s.mat,
+                   hv->cnt_part, reinterpret_cast<ulonglong2 *>(s.k[0]), flag);
+        count_launches(1);
+        end();
+    } else {
+        begin("q18_sort_hist");
+        launch_pdl(ob_hist_kernel, G, kObThreads, nb * 4, st, rows, amt, plan, nb, s.mat, s.big, 0, Q18PlanArgs{}, 0, flag);
+        count_launches(1);
+        end();
+    }
     begin("q18_sort_scan");
+    const bool tin = hv && kv_touch_mode() == 1;
     launch_pdl(ob_scan_kernel, (nb + 31) / 32, 32 * kScanWarps, 4 * std::max(32 * G, nb), st, s.mat, G, nb, s.count,
-               s.offset, s.ticket, (const Q18Plan *)plan);
+               s.offset, s.ticket, (const Q18Plan *)plan, tin ? reinterpret_cast<ulonglong2 *>(s.kv) : nullptr,
+               tin ? hv->n_o : (uint64_t)0);
     count_launches(1);
     end();
     begin("q18_dist_counts");
@@ -1489,9 +1846,21 @@ void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long lo
                (unsigned long long)out_cap);
     count_launches(1);
     end();
+    if (hv && kv_touch_mode() == 2) {
+        begin("q18_kv_touch");
+        launch_pdl(l2_touch_kernel, (unsigned)num_sms * 2, 1024, 0, st, reinterpret_cast<ulonglong2 *>(s.kv), hv->n_o,
+                   (const Q18Plan *)plan);
+        count_launches(1);
+        end();
+    }
     begin("q18_bucket_scatter");
-    launch_pdl(ob_scatter_kernel, G, kObThreads, nb * 4, st, rows, amt, (const Q18Plan *)plan, nb, (const unsigned int *)s.mat,
-               (const unsigned int *)s.offset, s.kv);
+    if (hv)
+        launch_pdl(ob_scatter_rec_kernel, G, kObThreads, nb * 4, st, reinterpret_cast<const ulonglong2 *>(s.k[0]),
+                   hv->n_o, (const Q18Plan *)plan, nb, (const unsigned int *)s.mat, (const unsigned int *)s.offset,
+                   (const unsigned int *)hv->cnt_part, reinterpret_cast<ulonglong2 *>(s.kv));
+    else
+        launch_pdl(ob_scatter_kernel, G, kObThreads, nb * 4, st, rows, amt, (const Q18Plan *)plan, nb,
+                   (const unsigned int *)s.mat, (const unsigned int *)s.offset, s.kv);
     count_launches(1);
     end();
     begin("q18_dist_send");
@@ -1499,6 +1868,7 @@ void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long lo
                reinterpret_cast<const ulonglong2 *>(s.kv), (const unsigned int *)s.offset, (const unsigned long long *)send);
     count_launches(1);
     end();
+    cudaMemsetAsync(s.big, 0, sizeof(unsigned int), st);  // the emit's oversized-bucket work list
     begin("q18_dist_wait");
     launch_peer_wait(pa, st);
     end();
@@ -1565,7 +1935,11 @@ cudaError_t set_attributes_sort(int num_sms) {
         (const void *)q18_dist_send_kernel,
         (const void *)q18_keys_hist_kernel,
         (const void *)q18_plan_kernel,
-        (const void *)scatter_kernel};
+        (const void *)scatter_kernel,
+        (const void *)q18_acc_stats_kernel,
+        (const void *)q18_having_rec_kernel,
+        (const void *)ob_scatter_rec_kernel,
+        (const void *)l2_touch_kernel};
     const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
     if (le != cudaSuccess) return le;
 
@@ -1581,6 +1955,8 @@ cudaError_t set_attributes_sort(int num_sms) {
         {(const void *)ob_scatter_kernel, 4 << kBucketMaxBits},
         {(const void *)ob_scan_kernel, 4 * std::max(32 * G, 1 << kBucketMaxBits)},
         {(const void *)q18_dist_route_kernel, 4 << kBucketMaxBits},
+        {(const void *)q18_having_rec_kernel, 4 << kBucketMaxBits},
+        {(const void *)ob_scatter_rec_kernel, 4 << kBucketMaxBits},
     };
     for (const auto &x : a) {
         const cudaError_t e = cudaFuncSetAttribute(x.f, cudaFuncAttributeMaxDynamicSharedMemorySize, x.bytes);
