@@ -560,7 +560,10 @@ template <int kLsCap> struct LsSmem {
     unsigned int v1[kLsCap], v2[kLsCap];
     unsigned int sub[kLsSubMax + 1];   // sub-bucket counts -> offsets
     unsigned int cur[kLsSubMax];       // sub-bucket cursors
-    unsigned int wsum[kEmThreads / 32];
+    // 16-byte aligned on its own: the compiler reads wsum[] with one 128-bit shared load, which
+    // from an unaligned start also covered the last cur[] entry — racecheck reported that benign
+    // over-read as a read/write hazard against the scan's cur[] stores
+    alignas(16) unsigned int wsum[kEmThreads / 32];
 };
 
 // carry mode: the records stay where they were loaded and the sort moves 16-bit record ids
@@ -571,7 +574,10 @@ template <int kCap> struct LcSmem {
     unsigned short srt[kCap];         // record ids in sorted order
     unsigned int sub[kLsSubMax + 1];
     unsigned int cur[kLsSubMax];
-    unsigned int wsum[kEmThreads / 32];
+    // 16-byte aligned on its own: the compiler reads wsum[] with one 128-bit shared load, which
+    // from an unaligned start also covered the last cur[] entry — racecheck reported that benign
+    // over-read as a read/write hazard against the scan's cur[] stores
+    alignas(16) unsigned int wsum[kEmThreads / 32];
 };
 static_assert(kLsCapLarge <= 65536, "16-bit record ids");
 constexpr int kLcCapLarge = 8192;  // carry records per bucket in the large instance (~172 KB)
