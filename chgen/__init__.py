@@ -66,7 +66,11 @@ TABLE_COLUMNS = {
                ("o_all_local", np.int32), ("o_entry_d", np.int64)],
     "customer": [("c_w_id", np.int32), ("c_d_id", np.int32), ("c_id", np.int32),
                  ("c_last", np.int32), ("c_state", "S2"), ("c_state_p2", np.int32)],
-    "new_order": [("no_w_id", np.int32), ("no_d_id", np.int32), ("no_o_id", np.int32)],
+    # no_deleted: 1 once a Delivery has deleted the row (TPC-C 2.7.4.2 DELETE FROM new_order), kept
+    # as an in-place update of a tombstone column so the device store stays append + update only
+    # (R35); every generated / inserted row has 0
+    "new_order": [("no_w_id", np.int32), ("no_d_id", np.int32), ("no_o_id", np.int32),
+                  ("no_deleted", np.int32)],
     "item": [("i_id", np.int32), ("i_price", np.int64), ("i_data", "S50"), ("i_data_p2", np.int32)],
 }
 
@@ -170,7 +174,7 @@ def _warehouse(w: int, seed: int, mode: str, sc: Scale):
     # district, NO_O_ID 2101..3000), in (d, o_id) order
     und = o_carrier == -1
     new_order = {"no_w_id": np.full(int(und.sum()), wi, dtype=np.int32), "no_d_id": o_d[und],
-                 "no_o_id": o_id[und]}
+                 "no_o_id": o_id[und], "no_deleted": np.zeros(int(und.sum()), dtype=np.int32)}
     return {"order_line": ol, "orders": orders, "customer": customer, "new_order": new_order}
 
 
@@ -309,7 +313,7 @@ def neworder_delta(state: NewOrderState, n_txn: int, *, seed: int, batch: int,
 def _new_order_rows(orders: dict) -> dict:
     """The new_order rows a NewOrder transaction inserts: one per new order (TPC-C 2.4.2.2)."""
     return {"no_w_id": orders["o_w_id"].astype(np.int32), "no_d_id": orders["o_d_id"].astype(np.int32),
-            "no_o_id": orders["o_id"].astype(np.int32)}
+            "no_o_id": orders["o_id"].astype(np.int32), "no_deleted": np.zeros(len(orders["o_id"]), np.int32)}
 
 
 def neworder_batch(state: NewOrderState, n_txn: int, *, seed: int, batch: int, item=None):
@@ -379,20 +383,23 @@ class DeliveryState:
     o_id order, each as (o_id, orders row, first order_line row, ol_cnt) — row positions in the
     host row store, which is what an in-place update names (NEXT-1).
 
-    ``add(orders, o_row0, ol_row0)`` registers a block of orders stored at orders rows
+    ``add(orders, o_row0, ol_row0, no_row0)`` registers a block of orders stored at orders rows
     ``o_row0 + i`` whose lines are stored contiguously, in the same order, from order_line row
-    ``ol_row0`` on (true for ``generate`` tables and for ``neworder_batch`` deltas)."""
+    ``ol_row0`` on (true for ``generate`` tables and for ``neworder_batch`` deltas); with
+    ``no_row0``, the k-th undelivered order of the block is new_order row ``no_row0 + k`` (true for
+    both as well: their new_order rows list the undelivered orders in orders-row order), which a
+    Delivery then deletes (a tombstone update of ``no_deleted``)."""
     districts: int = FULL.districts
     queues: dict = field(default_factory=dict)
 
-    def add(self, orders: dict, o_row0: int = 0, ol_row0: int = 0):
+    def add(self, orders: dict, o_row0: int = 0, ol_row0: int = 0, no_row0: int | None = None):
         cnt = orders["o_ol_cnt"].astype(np.int64)
         ol_first = ol_row0 + np.concatenate([[0], np.cumsum(cnt)[:-1]]) if len(cnt) else cnt
         pending = np.flatnonzero(orders["o_carrier_id"] == -1)
         w, d, o = orders["o_w_id"], orders["o_d_id"], orders["o_id"]
-        for i in pending.tolist():
+        for k, i in enumerate(pending.tolist()):
             self.queues.setdefault((int(w[i]), int(d[i])), deque()).append(
-                (int(o[i]), o_row0 + i, int(ol_first[i]), int(cnt[i])))
+                (int(o[i]), o_row0 + i, int(ol_first[i]), int(cnt[i]), -1 if no_row0 is None else no_row0 + k))
 
     def undelivered(self) -> int:
         return sum(len(q) for q in self.queues.values())
@@ -416,22 +423,27 @@ def delivery_batch(state: DeliveryState, w, carrier, clock0: int, step_us: int =
 
     Returns ``{"orders": {"o_carrier_id": (rows, values)},
     "order_line": {"ol_delivery_d": (rows, values)}}`` with rows uint32 (distinct: an order is
-    delivered once) and values in the column dtype."""
-    o_rows, o_vals, l_rows, l_vals = [], [], [], []
+    delivered once) and values in the column dtype; plus ``"new_order": {"no_deleted": (rows, 1s)}``
+    (the transaction's DELETE FROM new_order) for orders registered with their new_order row."""
+    o_rows, o_vals, l_rows, l_vals, n_rows = [], [], [], [], []
     for k in range(len(w)):
         ts = clock0 + (k + 1) * step_us
         for d in range(1, state.districts + 1):
             q = state.queues.get((int(w[k]), d))
             if not q:
                 continue
-            _, o_row, ol_first, cnt = q.popleft()
+            _, o_row, ol_first, cnt, no_row = q.popleft()
+            if no_row >= 0:
+                n_rows.append(no_row)
             o_rows.append(o_row)
             o_vals.append(int(carrier[k]))
             l_rows.extend(range(ol_first, ol_first + cnt))
             l_vals.extend([ts] * cnt)
-    return {"orders": {"o_carrier_id": (np.asarray(o_rows, np.uint32), np.asarray(o_vals, np.int32))},
-            "order_line": {"ol_delivery_d": (np.asarray(l_rows, np.uint32),
-                                             np.asarray(l_vals, np.int64))}}
+    out = {"orders": {"o_carrier_id": (np.asarray(o_rows, np.uint32), np.asarray(o_vals, np.int32))},
+           "order_line": {"ol_delivery_d": (np.asarray(l_rows, np.uint32), np.asarray(l_vals, np.int64))}}
+    if n_rows:
+        out["new_order"] = {"no_deleted": (np.asarray(n_rows, np.uint32), np.ones(len(n_rows), np.int32))}
+    return out
 
 
 # ------------------------------------------------------- NEXT-3 layout table --

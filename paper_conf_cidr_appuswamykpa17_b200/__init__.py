@@ -63,7 +63,8 @@ SCHEMA = {
         ("c_w_id", H2TAP_I32), ("c_d_id", H2TAP_I32), ("c_id", H2TAP_I32), ("c_last", H2TAP_I32),
         ("c_state_p2", H2TAP_I32)]),
     "item": (H2TAP_T_ITEM, [("i_id", H2TAP_I32), ("i_price", H2TAP_I64), ("i_data_p2", H2TAP_I32)]),
-    "new_order": (H2TAP_T_NEW_ORDER, [("no_w_id", H2TAP_I32), ("no_d_id", H2TAP_I32), ("no_o_id", H2TAP_I32)]),
+    "new_order": (H2TAP_T_NEW_ORDER, [("no_w_id", H2TAP_I32), ("no_d_id", H2TAP_I32), ("no_o_id", H2TAP_I32),
+                                      ("no_deleted", H2TAP_I32)]),
 }
 
 
@@ -563,7 +564,7 @@ def plan_columns():
         H2TAP_Q3: {"order_line": ["ol_w_id", "ol_d_id", "ol_o_id", "ol_amount"],
                    "orders": ["o_w_id", "o_d_id", "o_id", "o_c_id", "o_ol_cnt", "o_entry_d"],
                    "customer": ["c_w_id", "c_d_id", "c_id", "c_state_p2"],
-                   "new_order": ["no_w_id", "no_d_id", "no_o_id"]},
+                   "new_order": ["no_w_id", "no_d_id", "no_o_id", "no_deleted"]},
         H2TAP_Q6: {"order_line": ["ol_delivery_d", "ol_quantity", "ol_amount"]},
         H2TAP_Q1: {"order_line": ["ol_number", "ol_delivery_d", "ol_quantity", "ol_amount"]},
         H2TAP_Q18: {"order_line": ["ol_w_id", "ol_d_id", "ol_o_id", "ol_amount"],
@@ -582,7 +583,12 @@ def hot_path_tables(tables: dict, plans=HOT_PATH_PLANS) -> dict:
             for c in cols:
                 if c not in want[t]:
                     want[t].append(c)
-    return {t: {c: tables[t][c] for c in cols} for t, cols in want.items()}
+    # optional columns (new_order.no_deleted: Delivery's tombstones) are taken when present
+    return {t: {c: tables[t][c] for c in cols if c in tables[t] or (t, c) not in OPTIONAL_COLUMNS}
+            for t, cols in want.items()}
+
+
+OPTIONAL_COLUMNS = {("new_order", "no_deleted")}
 
 
 def h2tap_layout_sum(engine: Engine, data, layout: int, nrows: int, ncols: int, columns, *,

@@ -79,14 +79,14 @@ struct Fail {  // thrown internally, converted to a status at the ABI boundary
 // ============================================================== schema ===
 constexpr int kTables = 6;  // index = table id (1..5)
 constexpr int kMaxCols = 9;
-const int kNcols[kTables] = {0, 9, 8, 5, 3, 3};
+const int kNcols[kTables] = {0, 9, 8, 5, 3, 4};
 const uint32_t kTypes[kTables][kMaxCols] = {
     {},
     {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64},
     {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64},
     {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32},
     {H2TAP_I32, H2TAP_I64, H2TAP_I32},
-    {H2TAP_I32, H2TAP_I32, H2TAP_I32}};
+    {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I32}};
 inline size_t type_size(uint32_t t) { return t == H2TAP_I32 ? 4 : 8; }
 constexpr uint64_t kPadRows = 64;  // over-allocation so 128-bit loads of the last tile stay in bounds
 
@@ -1445,7 +1445,7 @@ void launch_q3_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     e->prof.run("q3_mark", [&] {
         if (n_no)
             launch_q3_mark(colp<int32_t>(v, NO, H2TAP_NO_W_ID), colp<int32_t>(v, NO, H2TAP_NO_D_ID),
-                           colp<int32_t>(v, NO, H2TAP_NO_O_ID), n_no, colp<int32_t>(v, O, H2TAP_O_W_ID),
+                           colp<int32_t>(v, NO, H2TAP_NO_O_ID), colp<int32_t>(v, NO, H2TAP_NO_DELETED), n_no, colp<int32_t>(v, O, H2TAP_O_W_ID),
                            colp<int32_t>(v, O, H2TAP_O_D_ID), colp<int32_t>(v, O, H2TAP_O_C_ID),
                            colp<int64_t>(v, O, H2TAP_O_ENTRY_D), colp<int32_t>(v, C, H2TAP_C_STATE_P2),
                            q.p[0], (int)q.p[1], s, e->num_sms, e->compute);

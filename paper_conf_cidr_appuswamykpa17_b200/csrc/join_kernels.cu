@@ -401,7 +401,7 @@ __device__ __forceinline__ bool like_prefix2(int p2, int prefix) {
 }
 
 __global__ void q3_mark_kernel(const int32_t *__restrict__ no_w, const int32_t *__restrict__ no_d,
-                               const int32_t *__restrict__ no_o, uint64_t n_no,
+                               const int32_t *__restrict__ no_o, const int32_t *__restrict__ no_del, uint64_t n_no,
                                const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
                                const int32_t *__restrict__ o_c, const int64_t *__restrict__ o_ent,
                                const int32_t *__restrict__ c_p2, long long entry_lo, int prefix,
@@ -411,7 +411,9 @@ __global__ void q3_mark_kernel(const int32_t *__restrict__ no_w, const int32_t *
     const uint64_t n_pad = (n_no + 31) & ~31ull;  // whole warps iterate together (ballot below)
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n_pad; i += stride) {
         unsigned int orow = kNoRow;
-        if (i < n_no) orow = jx_lookup(s.jo, __ldcs(no_w + i), __ldcs(no_d + i), __ldcs(no_o + i));
+        // a deleted new_order row (Delivery's DELETE, a tombstone update) is not there: no join
+        if (i < n_no && !(no_del && __ldcs(no_del + i)))
+            orow = jx_lookup(s.jo, __ldcs(no_w + i), __ldcs(no_d + i), __ldcs(no_o + i));
         bool hit = false;
         if (orow != kNoRow && __ldg(o_ent + orow) > entry_lo) {
             const unsigned int crow = jx_lookup(s.jc, __ldg(o_w + orow), __ldg(o_d + orow), __ldg(o_c + orow));
@@ -527,11 +529,11 @@ void launch_q18_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *o
     count_launches(1);
 }
 
-void launch_q3_mark(const int32_t *no_w, const int32_t *no_d, const int32_t *no_o, uint64_t n_no,
+void launch_q3_mark(const int32_t *no_w, const int32_t *no_d, const int32_t *no_o, const int32_t *no_del, uint64_t n_no,
                     const int32_t *o_w, const int32_t *o_d, const int32_t *o_c, const int64_t *o_ent,
                     const int32_t *c_p2, int64_t entry_lo, int prefix, const Q18Scratch &s, int num_sms,
                     cudaStream_t st) {
-    q3_mark_kernel<<<grid_for(n_no, 256, num_sms, 8), 256, 0, st>>>(no_w, no_d, no_o, n_no, o_w, o_d, o_c,
+    q3_mark_kernel<<<grid_for(n_no, 256, num_sms, 8), 256, 0, st>>>(no_w, no_d, no_o, no_del, n_no, o_w, o_d, o_c,
                                                                  o_ent, c_p2, entry_lo, prefix, s);
     count_launches(1);
 }

@@ -175,7 +175,8 @@ void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_
 // CH Q3 (NEXT-2) on the Q18 machinery: mark orders rows joined by new_order and an 'prefix%'
 // customer (multiplicity in acc[].pad, candidate list in cand / *ncand), probe order_line into the
 // marked rows only, emit result rows (revenue = sum x multiplicity, count *nout) + sort statistics.
-void launch_q3_mark(const int32_t *no_w, const int32_t *no_d, const int32_t *no_o, uint64_t n_no,
+// no_del: the new_order tombstone column (null: no row deleted); deleted rows join nothing
+void launch_q3_mark(const int32_t *no_w, const int32_t *no_d, const int32_t *no_o, const int32_t *no_del, uint64_t n_no,
                     const int32_t *o_w, const int32_t *o_d, const int32_t *o_c, const int64_t *o_ent,
                     const int32_t *c_p2, int64_t entry_lo, int prefix, const Q18Scratch &s, int num_sms,
                     cudaStream_t st);

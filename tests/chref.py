@@ -78,7 +78,7 @@ def sqlite_load(tables):
         db.executemany("UPDATE customer SET c_state = ? WHERE rowid = ?",
                        [(bytes(x).decode("latin-1"), i + 1) for i, x in enumerate(c["c_state"])])
     if "new_order" in tables:
-        no = tables["new_order"]
+        no = live_new_order(tables["new_order"])
         db.execute("CREATE TABLE new_order (no_w_id INT, no_d_id INT, no_o_id INT)")
         db.executemany("INSERT INTO new_order VALUES (?,?,?)",
                        zip(no["no_w_id"].tolist(), no["no_d_id"].tolist(), no["no_o_id"].tolist()))
@@ -157,16 +157,38 @@ def sqlite_q3(db, entry_lo, prefix="A"):
 def sqlite_delivery(db, w, carrier, ts, districts):
     """One TPC-C Delivery transaction (TPC-C 2.7.4.2 [EXT]) as SQL: for each district, the
     oldest undelivered order (new_order = orders with a NULL carrier) gets the carrier and its
-    lines get delivery date ts."""
+    lines get delivery date ts, and (when the database holds new_order) its new_order row is
+    deleted."""
+    has_no = db.execute("SELECT name FROM sqlite_master WHERE name = 'new_order'").fetchone() is not None
     for d in range(1, districts + 1):
         (o,) = db.execute("SELECT MIN(o_id) FROM orders WHERE o_w_id = ? AND o_d_id = ? "
                           "AND o_carrier_id IS NULL", (w, d)).fetchone()
         if o is None:
             continue
+        if has_no:
+            db.execute("DELETE FROM new_order WHERE no_w_id = ? AND no_d_id = ? AND no_o_id = ?", (w, d, o))
         db.execute("UPDATE orders SET o_carrier_id = ? WHERE o_w_id = ? AND o_d_id = ? AND o_id = ?",
                    (carrier, w, d, o))
         db.execute("UPDATE order_line SET ol_delivery_d = ? "
                    "WHERE ol_w_id = ? AND ol_d_id = ? AND ol_o_id = ?", (ts, w, d, o))
+
+
+def live_new_order(no):
+    """The new_order rows a query sees: those without a Delivery tombstone (no_deleted = 1 is the
+    device store's record of DELETE FROM new_order, R35) — the plain definition of a
+    deleted row, which simply is not there."""
+    if "no_deleted" not in no:
+        return no
+    keep = np.asarray(no["no_deleted"]) == 0
+    return {c: np.asarray(v)[keep] for c, v in no.items() if c != "no_deleted"}
+
+
+def visible(tables):
+    """A table set as SQL sees it: deleted new_order rows removed."""
+    out = dict(tables)
+    if "new_order" in out:
+        out["new_order"] = live_new_order(out["new_order"])
+    return out
 
 
 def sqlite_column(db, table, column, null):

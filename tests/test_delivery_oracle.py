@@ -15,7 +15,7 @@ import pytest
 import chgen
 import oracle
 from chref import (Q18_HAVING, sqlite_column, sqlite_delivery, sqlite_load, sqlite_q1,
-                   sqlite_q18, sqlite_q6)
+                   sqlite_q18, sqlite_q3, sqlite_q6, visible)
 
 NULL = np.iinfo(np.int64).min
 
@@ -106,3 +106,47 @@ def test_delivery_takes_oldest_order_per_district():
         {(d, sc.delivered_below) for d in range(1, sc.districts + 1)}
     assert len(lrows) == int(o["o_ol_cnt"][rows].sum())
     assert (lvals == chgen.TS_2025 + 1000).all()
+
+
+def test_delivery_deletes_new_order_rows_like_sqlite():
+    """Delivery's DELETE FROM new_order as a tombstone update (R35): SQLite executes
+    the DELETE; the new_order rows without a tombstone in chgen's updated snapshot must be exactly
+    SQLite's remaining rows (rowid order), and CH Q3 — which joins new_order — must agree between
+    SQLite and the oracle on the visible snapshot, epoch after epoch, across a NewOrder delta."""
+    sc = chgen.TINY
+    W = 2
+    t = chgen.generate(1, W + 1, seed=15, scale=sc)
+    item = t.pop("item")
+    st = chgen.DeliveryState(districts=sc.districts)
+    st.add(t["orders"], 0, 0, 0)  # generated new_order rows list the undelivered orders in order
+    no = chgen.NewOrderState(1, W + 1, scale=sc)
+    delta = chgen.neworder_batch(no, 10, seed=15, batch=0, item=item)
+    st.add(delta["orders"], len(t["orders"]["o_id"]), len(t["order_line"]["ol_o_id"]),
+           len(t["new_order"]["no_o_id"]))
+    for tb in ("orders", "order_line", "new_order"):
+        t[tb] = {c: np.concatenate([t[tb][c], delta[tb][c]]) for c in t[tb]}
+    db = sqlite_load(t)
+    snap = t
+    clock = chgen.TS_2025 + 3 * chgen.DAY_US
+    entry_lo = chgen.TS_1995
+    deleted = 0
+    for b in range(5):
+        w, carrier = chgen.delivery_inputs(2, seed=15, batch=b, w_lo=1, w_hi=W + 1)
+        upd = chgen.delivery_batch(st, w, carrier, clock)
+        for k in range(len(w)):
+            sqlite_delivery(db, int(w[k]), int(carrier[k]), clock + (k + 1) * 1000, sc.districts)
+        clock += len(w) * 1000
+        snap = oracle.apply_updates(snap, upd)
+        deleted += len(upd["new_order"]["no_deleted"][0])
+        vis = visible(snap)["new_order"]
+        got = db.execute("SELECT no_w_id, no_d_id, no_o_id FROM new_order ORDER BY rowid").fetchall()
+        assert got == list(zip(vis["no_w_id"].tolist(), vis["no_d_id"].tolist(), vis["no_o_id"].tolist()))
+        assert int(snap["new_order"]["no_deleted"].sum()) == deleted > 0
+        want = sqlite_q3(db, entry_lo, "")
+        got3 = oracle.q3(visible(snap), entry_lo, b"")
+        rows = list(zip(got3["ol_o_id"].tolist(), got3["ol_w_id"].tolist(), got3["ol_d_id"].tolist(),
+                        got3["revenue"].tolist(), got3["o_entry_d"].tolist()))
+        assert len(rows) > 0
+        # SQLite breaks ORDER BY ties arbitrarily: the ordered sort keys and the row set must match
+        assert [(r[3], r[4]) for r in rows] == [(r[3], r[4]) for r in want]
+        assert sorted(rows) == sorted(tuple(r) for r in want)

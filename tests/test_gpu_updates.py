@@ -308,3 +308,59 @@ def test_full_size_w100_delivery_epoch(h):
         assert st["cow_full_copies"] == 1 and st["cow_pages_copied"] > 0
     finally:
         h.h2tap_close(e)
+
+
+def test_delivery_deletes_new_order_rows_q3(h):
+    """Delivery's DELETE FROM new_order on the device store (R35): a tombstone update of
+    new_order.no_deleted, copy-on-write like every update, published with the epoch's appends
+    (NewOrder inserts orders, lines AND new_order rows). CH Q3 — the query that joins new_order —
+    must equal the oracle on the visible snapshot (deleted rows removed; pinned to SQLite's
+    DELETE in test_delivery_oracle.py) epoch after epoch, with no reload of new_order."""
+    from chref import visible
+    from test_oracle_q3 import Q3_LO
+    W, seed = 2, 57
+    plans = (h.H2TAP_Q3, h.H2TAP_Q18)
+    snap = chgen.generate(1, W + 1, seed=seed)
+    item = snap.pop("item")
+    dl = chgen.DeliveryState()
+    dl.add(snap["orders"], 0, 0, 0)
+    no = chgen.NewOrderState(1, W + 1)
+    e = h.h2tap_open(0)
+    try:
+        epoch = 1
+        h.h2tap_load_snapshot(e, h.hot_path_tables(snap, plans), epoch)
+        clock = chgen.TS_2025 + 5 * chgen.DAY_US
+        lo = chgen.TS_1995
+        deleted = 0
+        for b in range(4):
+            n_o, n_ol, n_no = (len(snap["orders"]["o_id"]), len(snap["order_line"]["ol_o_id"]),
+                               len(snap["new_order"]["no_o_id"]))
+            delta = chgen.neworder_batch(no, 200, seed=seed, batch=b, item=item)
+            dl.add(delta["orders"], n_o, n_ol, n_no)
+            w, carrier = chgen.delivery_inputs(30, seed=seed, batch=b, w_lo=1, w_hi=W + 1)
+            upd = chgen.delivery_batch(dl, w, carrier, clock)
+            clock += 31_000
+            deleted += len(upd["new_order"]["no_deleted"][0])
+            grown = {t: (_concat(snap[t], delta[t]) if t in delta else snap[t]) for t in snap}
+            snap = oracle.apply_updates(grown, upd)
+            epoch += 1
+            dev = h.hot_path_tables({**delta, "customer": snap["customer"]}, plans)
+            dev.pop("customer")
+            dev_upd = {"new_order": upd["new_order"]}  # Q3/Q18 read no other updated column
+            h.h2tap_refresh(e, dev, dev_upd, epoch, first_row={"orders": n_o, "order_line": n_ol, "new_order": n_no})
+            for prefix in (b"A", b""):
+                code = (prefix[0] << 8) if prefix else 0
+                r = h.h2tap_run_query(e, h.H2TAP_Q3, [lo, code])
+                got = r.to_numpy()
+                r.free()
+                want = oracle.q3(visible(snap), lo, prefix)
+                for k in want:
+                    assert np.array_equal(got[k], want[k]), (b, prefix, k)
+            # the tombstones matter: with the deleted rows still there Q3 would differ
+            assert len(oracle.q3(snap | {"new_order": {c: v for c, v in snap["new_order"].items()
+                                                        if c != "no_deleted"}}, lo, b"")["ol_o_id"]) > \
+                len(oracle.q3(visible(snap), lo, b"")["ol_o_id"])
+        assert deleted > 0
+        assert h.h2tap_get_store_stats(e)["rows_updated"] >= deleted
+    finally:
+        h.h2tap_close(e)
