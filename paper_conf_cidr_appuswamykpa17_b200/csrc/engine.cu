@@ -386,6 +386,12 @@ struct h2tap_engine {
         bool connected = false, broken = false;
     } peer;
     cudaStream_t compute = nullptr, copy = nullptr;
+    // H2TAP_Q18_STREAM=1: a batch's Q18 / Q3 run on this second compute stream, forked from the
+    // batch start and joined before the batch's host synchronisation, so their latency-bound
+    // kernels can overlap the bandwidth-bound scans of the other queries
+    cudaStream_t side = nullptr;
+    bool q18_side = false;
+    cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
     cudaStream_t reaper = nullptr;  // stream-ordered frees of snapshot buffers
     FreeOrder free_order;
     cudaEvent_t q_begin = nullptr, q_end = nullptr;
@@ -1848,7 +1854,10 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
         ~Cleanup() {
             bool pending = false;
             for (auto &q : c) pending |= !q.dev_blocks.empty() || q.small.first;
-            if (pending) cudaStreamSynchronize(e->compute);  // kernels may still use the blocks
+            if (pending) {  // kernels may still use the blocks
+                cudaStreamSynchronize(e->side);
+                cudaStreamSynchronize(e->compute);
+            }
             for (auto &q : c) {
                 release_dev_blocks(e, q);
                 if (q.small.first) e->host_pool->put(q.small.first, q.small.second);
@@ -1858,8 +1867,16 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
     // launch phase: a plan's scratch is reused by a later query of the same plan, so a repeated
     // plan first completes the queries launched before it
     size_t done = 0;
+    bool forked = false;
+    auto join_side = [&] {
+        if (!forked) return;
+        CK(cudaEventRecord(e->ev_join, e->side));
+        CK(cudaStreamWaitEvent(e->compute, e->ev_join, 0));
+        forked = false;
+    };
     auto finish_upto = [&](size_t upto) {
         if (done >= upto) return;
+        join_side();
         sync_compute(e);
         if (e->world > 1 && *reinterpret_cast<volatile unsigned int *>(e->peer.err_host)) {
             e->peer.broken = true;
@@ -1879,6 +1896,7 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
             }
         }
     };
+    CK(cudaEventRecord(e->ev_fork, e->compute));  // the batch start (fork point of the side stream)
     for (size_t i = 0; i < ctx.size(); ++i) {
         QueryCtx &q = ctx[i];
         for (size_t j = done; j < i; ++j)
@@ -1892,6 +1910,23 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
         }
         q.mark0 = e->prof.marks.size();
         q.launches0 = launches_total();
+        // Q18 / Q3 on the side stream (only when something else in the batch could overlap)
+        const bool on_side = e->q18_side && n > 1 && (q.plan == H2TAP_Q18 || q.plan == H2TAP_Q3);
+        if (on_side && !forked) {  // fork from the batch start: the side work need not wait for
+                                   // the queries enqueued before it on the compute stream
+            CK(cudaStreamWaitEvent(e->side, e->ev_fork, 0));
+            forked = true;
+        }
+        struct SideSwap {  // launch this query's work on the side stream (scratch ordered there)
+            h2tap_engine *e; bool on;
+            SideSwap(h2tap_engine *x, bool o) : e(x), on(o) { if (on) swap(); }
+            ~SideSwap() { if (on) swap(); }
+            void swap() {
+                std::swap(e->compute, e->side);
+                e->arena.owner = e->compute;
+                e->prof.st = e->compute;
+            }
+        } side_swap(e, on_side);
         CK(cudaEventRecord(q.begin, e->compute));
         switch (q.plan) {
             case H2TAP_Q1: launch_q1_plan(e, *v, q); break;
@@ -1906,6 +1941,7 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
         q.launches = launches_total() - q.launches0;
         q.mark1 = e->prof.marks.size();
     }
+    join_side();
     finish_upto(ctx.size());
     const double wall = std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - t0).count();
     for (uint32_t i = 0; i < n; ++i) {
@@ -1997,6 +2033,10 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
 
         CK(cudaStreamCreateWithFlags(&e->compute, cudaStreamNonBlocking));
         CK(cudaStreamCreateWithFlags(&e->copy, cudaStreamNonBlocking));
+        CK(cudaStreamCreateWithFlags(&e->side, cudaStreamNonBlocking));
+        CK(cudaEventCreateWithFlags(&e->ev_fork, cudaEventDisableTiming));
+        CK(cudaEventCreateWithFlags(&e->ev_join, cudaEventDisableTiming));
+        if (const char *q = std::getenv("H2TAP_Q18_STREAM")) e->q18_side = std::atoi(q) != 0;
         CK(cudaStreamCreateWithFlags(&e->reaper, cudaStreamNonBlocking));
         e->free_order = FreeOrder{e->compute, e->copy, e->reaper};
         {   // keep freed pool memory cached (no release to the OS at stream syncs)
@@ -2304,6 +2344,10 @@ void h2tap_close(h2tap_engine *e) {
     cudaStreamSynchronize(e->reaper);
     cudaStreamDestroy(e->compute);
     cudaStreamDestroy(e->copy);
+    cudaStreamSynchronize(e->side);
+    cudaStreamDestroy(e->side);
+    cudaEventDestroy(e->ev_fork);
+    cudaEventDestroy(e->ev_join);
     cudaStreamDestroy(e->reaper);
     delete e;
 }

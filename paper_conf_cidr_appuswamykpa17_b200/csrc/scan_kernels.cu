@@ -8,6 +8,7 @@
 // (L527-535) with fusion as future work (L552-554): here each query is ONE fused kernel plus a
 // tiny finaliser, and the scan is HBM-bound (20 B/row for Q6, 24 B/row for Q1).
 #include <algorithm>
+#include <cstdlib>
 #include <cstdint>
 #include <cuda_runtime.h>
 
@@ -769,11 +770,18 @@ void launch_q6(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uin
         count_launches(1);
 }
 
+// SMs the TMA scans use (H2TAP_SCAN_SMS, A/B: a scan on part of the GPU, the rest free for
+// concurrent work)
+int scan_sms(int num_sms) {
+    static const int lim = [] { const char *v = std::getenv("H2TAP_SCAN_SMS"); return v ? std::atoi(v) : 0; }();
+    return lim > 0 && lim < num_sms ? lim : num_sms;
+}
+
 void launch_q6_tma(const int64_t *deliv, const int32_t *qty, const int64_t *amt, uint64_t n,
                    int64_t d_lo, int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s,
                    int num_sms, cudaStream_t st) {
     const uint64_t nchunks = (n + kQ6Chunk - 1) / kQ6Chunk;
-    const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
+    const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)scan_sms(num_sms)));
     launch_pdl(q6_tma_kernel, grid, kTmaThreads, sizeof(Q6TmaSmem), st,
         reinterpret_cast<const long long *>(deliv), qty, reinterpret_cast<const long long *>(amt), n,
         Q6Pred{d_lo, d_hi, q_lo, q_hi}, s.block_part, s.done_counter, s.out, s.host_out);
@@ -807,7 +815,7 @@ void launch_q1_tma(const int32_t *number, const int64_t *deliv, const int32_t *q
     using Cfg = Q1TmaCfg<false>;
     const size_t smem = sizeof(Q1StagesT<Cfg::kS>) + sizeof(Q1SmemT<Cfg::kT>);
     const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
-    const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
+    const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)scan_sms(num_sms)));
     launch_pdl(q1_tma_kernel<false>, grid, (Q1TmaCfg<false>::kW + 1) * 32, smem, st, number, reinterpret_cast<const long long *>(deliv), qty,
                reinterpret_cast<const long long *>(amt), n, cutoff, s, Q6Pred{0, 0, 0, 0}, nullptr, nullptr,
                nullptr, nullptr);
@@ -821,7 +829,7 @@ void launch_q61_tma(const int32_t *number, const int64_t *deliv, const int32_t *
     using Cfg = Q1TmaCfg<true>;
     const size_t smem = sizeof(Q1StagesT<Cfg::kS>) + sizeof(Q1SmemT<Cfg::kT>);
     const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
-    const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)num_sms));
+    const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)scan_sms(num_sms)));
     launch_pdl(q1_tma_kernel<true>, grid, kQ61Threads, smem, st, number, reinterpret_cast<const long long *>(deliv),
                qty, reinterpret_cast<const long long *>(amt), n, cutoff, s, Q6Pred{d_lo, d_hi, q_lo, q_hi},
                s6.block_part, s6.done_counter, s6.out, s6.host_out);
