@@ -71,13 +71,15 @@ if traffic:
              "bucket_local_emit_kernel<2048, 0, 1>": "q18_bucket_sort_emit",
              "bucket_local_emit_kernel<8192, 2048, 1>": "q18_bucket_sort_emit_large",
              "q18_plan_kernel": "q18_plan", "q1_compact_kernel": "q1_compact",
-             "q1_emit_kernel": "q1_emit"}
+             "q1_emit_kernel": "q1_emit", "q1_tma_kernel<1>": "q61_shared_scan",
+             "q18_acc_stats_kernel": "q18_acc_stats", "q18_having_rec_kernel": "q18_having_records",
+             "ob_scatter_rec_kernel": "q18_bucket_scatter"}
     bymark = {}
     for k, v in per.items():
         m = marks.get(k)
         if m:
             bymark[m] = bymark.get(m, 0.0) + v
     if len(sys.argv) > 2 and sys.argv[2] == "--bench":
-        json.dump({"source": f"profiles/{tag}_ncu_summary.md (ncu --set full, per launch)",
+        json.dump({"source": f"profiles/{tag}_ncu_summary.md (ncu --set full, per launch, dram read + write)",
                    **{k: int(v) for k, v in bymark.items()}},
                   open(os.path.join(root, "profiles", "ncu_traffic.json"), "w"), indent=1)
