@@ -73,7 +73,9 @@ if traffic:
              "q18_plan_kernel": "q18_plan", "q1_compact_kernel": "q1_compact",
              "q1_emit_kernel": "q1_emit", "q1_tma_kernel<1>": "q61_shared_scan",
              "q18_acc_stats_kernel": "q18_acc_stats", "q18_having_rec_kernel": "q18_having_records",
-             "ob_scatter_rec_kernel": "q18_bucket_scatter"}
+             "ob_scatter_rec_kernel": "q18_bucket_scatter",
+             "bucket_local_emit_kernel<1536, 0, 1>": "q18_bucket_sort_emit",
+             "bucket_local_emit_kernel<8192, 1536, 1>": "q18_bucket_sort_emit_large"}
     bymark = {}
     for k, v in per.items():
         m = marks.get(k)
