@@ -58,6 +58,8 @@ def parse():
                     help="strong scaling: this many warehouses split over the GPUs (config C4)")
     ap.add_argument("--peer-heap-mb", type=int, default=0, help="world > 1: peer heap per rank (0 = 1 GiB)")
     ap.add_argument("--no-c1", action="store_true", help="skip the config C1 line (Q6 at W=1)")
+    ap.add_argument("--plans", default="q6,q1,q18",
+                    help="the step's queries (config C4 is Q1 + Q6: --plans q6,q1)")
     ap.add_argument("--mode", default="spread", choices=["spread", "strict"])
     ap.add_argument("--e2e-steps", type=int, default=None)
     ap.add_argument("--no-cpu-baseline", action="store_true")
@@ -434,7 +436,9 @@ def main():
             dist.all_reduce(t, op=dist.ReduceOp.MAX)
         return [float(x) for x in t.tolist()]
 
-    plans = (("q6", h.H2TAP_Q6, Q6_P), ("q1", h.H2TAP_Q1, Q1_P), ("q18", h.H2TAP_Q18, Q18_P))
+    want = [x.strip() for x in a.plans.split(",") if x.strip()]
+    plans = tuple(p for p in (("q6", h.H2TAP_Q6, Q6_P), ("q1", h.H2TAP_Q1, Q1_P), ("q18", h.H2TAP_Q18, Q18_P))
+                  if p[0] in want)
 
     def run_batch(sel, flags):
         rs = h.h2tap_run_queries(eng, [(plan, p, flags) for name, plan, p in plans if name in sel])
@@ -450,7 +454,7 @@ def main():
     dense_seen = []
     dev_flags = h.H2TAP_RESULT_DEVICE
     prof_flags = h.H2TAP_RESULT_DEVICE | h.H2TAP_QUERY_PROFILE
-    ALL = ("q6", "q1", "q18")
+    ALL = tuple(p[0] for p in plans)
     clocks = Clocks(local)  # sampled from warm-up to the end of the instrumented pass
     time.sleep(0.3)
     for _ in range(a.warmup):
@@ -466,7 +470,7 @@ def main():
     # ---- timed region: K steps, CUDA events on the engine's stream, no per-kernel instrumentation
     starts = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
     ends = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
-    per_query = {"q6": [], "q1": [], "q18": []}
+    per_query = {q: [] for q in ALL}
     launches = 0
     n_pass = n_pass_total = 0
     barrier()
@@ -480,7 +484,8 @@ def main():
         for q, (ms, ks, nrows, nl, tot) in out.items():
             per_query[q].append(ms)
             launches += nl
-        n_pass, n_pass_total = out["q18"][2], out["q18"][4]
+        if "q18" in out:
+            n_pass, n_pass_total = out["q18"][2], out["q18"][4]
     barrier()
     step_ms_local = sum(s.elapsed_time(e) for s, e in zip(starts, ends)) / a.steps
 
@@ -489,7 +494,7 @@ def main():
     # kernels); a ~50 us sleep kernel queued first lets the host enqueue the whole query before the
     # GPU reaches it, so no launch latency lands inside the window
     alone = {}
-    for q in ("q6", "q1"):
+    for q in [x for x in ("q6", "q1") if x in ALL]:
         for _ in range(2):
             run_batch((q,), dev_flags)
         barrier()
@@ -513,7 +518,8 @@ def main():
                 kern.setdefault(kname, []).append(kms)
     barrier()
     clk = clocks.stop()
-    step_ms, q6_alone_ms, q1_alone_ms = max_over_ranks([step_ms_local, alone["q6"], alone["q1"]])
+    step_ms, q6_alone_ms, q1_alone_ms = max_over_ranks([step_ms_local, alone.get("q6", float("nan")),
+                                                       alone.get("q1", float("nan"))])
     lat = {q: float(np.median(v)) for q, v in per_query.items()}
     lat_max = dict(zip(lat, max_over_ranks(list(lat.values()))))
     nt = torch.tensor([n_ol], dtype=torch.float64, device="cuda")
@@ -618,15 +624,16 @@ def main():
             "warmup": a.warmup, "ms_per_step": step_ms, "higher_is_better": True,
             "scaling": "strong" if strong else "weak", "vs_baseline": None, "dtype": "int64",
             "data": "synthetic",
-            "config": {"workload": (f"CH Q6+Q1+Q18 per step over W={W} warehouses split over {world} GPU(s)"
+            "config": {"workload": (f"CH {'+'.join(q.upper() for q in ALL)} per step over W={W} warehouses split over {world} GPU(s)"
                                     if strong else
-                                    f"CH Q6+Q1+Q18 per step over W={a.warehouses} warehouses per GPU")
+                                    f"CH {'+'.join(q.upper() for q in ALL)} per step over W={a.warehouses} warehouses per GPU")
                                    + f" ('{a.mode}' TPC-C population, seed 1)",
                        "warehouses_total": W, "warehouses_per_gpu": W / world,
                        "order_line_rows_total": rows_total, "order_line_rows_rank0": n_ol,
                        "orders_rows_rank0": n_o, "customer_rows_rank0": n_c,
-                       "rows_counted": ROWS_COUNTED,
-                       "queries_per_step": 3, "parallelism": f"row-sharded by warehouse x{world}",
+                       "rows_counted": ("each visible order_line row counted once per step; one step = CH "
+                                        + " + ".join(q.upper() for q in ALL) + " over the snapshot"),
+                       "queries_per_step": len(ALL), "parallelism": f"row-sharded by warehouse x{world}",
                        "merge": ("peer-memory kernels over NVLink (Q6 allreduce, Q1 group lists, Q18 "
                                  "range-partitioned ORDER BY; DESIGN.md §6)" if world > 1 else "none (1 GPU)"),
                        "scan_sharing": ("Q6 and Q1 of the batch share one pass over order_line "
@@ -636,14 +643,12 @@ def main():
                                         if os.environ.get("H2TAP_SHARED_SCAN", "1") != "0" else "off"),
                        "l2": ("inputs > L2; between steps (outside events) 512 MB written then 256 MB read to flush L2"
                               if flush is not None else "inputs > L2 (no flush)")},
-            "latency_ms": {"q6_q1_shared_scan_batch": round(lat_max["q6"] + lat_max["q1"], 4),
-                           "q6_in_batch": round(lat_max["q6"], 4), "q1_in_batch": round(lat_max["q1"], 4),
-                           "q18": round(lat_max["q18"], 4),
-                           "q6_alone": round(q6_alone_ms, 4), "q1_alone": round(q1_alone_ms, 4)},
-            "rows_per_s": {"q6_alone": rows_total / (q6_alone_ms / 1e3),
-                           "q1_alone": rows_total / (q1_alone_ms / 1e3),
-                           "q6_q1_batch": rows_total / ((lat_max["q6"] + lat_max["q1"]) / 1e3),
-                           "q18": rows_total / (lat_max["q18"] / 1e3)},
+            "latency_ms": dict({f"{q}_in_batch": round(v, 4) for q, v in lat_max.items()},
+                               q6_alone=round(q6_alone_ms, 4), q1_alone=round(q1_alone_ms, 4),
+                               **({"q6_q1_shared_scan_batch": round(lat_max["q6"] + lat_max["q1"], 4)}
+                                  if "q6" in lat_max and "q1" in lat_max else {})),
+            "rows_per_s": dict({f"{q}_in_batch": rows_total / (v / 1e3) for q, v in lat_max.items()},
+                               q6_alone=rows_total / (q6_alone_ms / 1e3), q1_alone=rows_total / (q1_alone_ms / 1e3)),
             "q18_result_rows_total": n_pass_total, "q18_result_rows_rank0": n_pass,
             "roofline": roof,
             "kernels": kernels_summary,
