@@ -568,16 +568,16 @@ template <int kLsCap> struct LsSmem {
 
 // carry mode: the records stay where they were loaded and the sort moves 16-bit record ids
 // (1 536 rows: 35 KB, 6 blocks of 128 threads per SM)
-template <int kCap> struct LcSmem {
+template <int kCap, int kSub = kLsSubMax, int kT = kEmThreads> struct LcSmem {
     ulonglong2 rec[kCap];             // the bucket's records, load order
     unsigned short idx[kCap];         // record ids grouped by sub-bucket
     unsigned short srt[kCap];         // record ids in sorted order
-    unsigned int sub[kLsSubMax + 1];
-    unsigned int cur[kLsSubMax];
+    unsigned int sub[kSub + 1];
+    unsigned int cur[kSub];
     // 16-byte aligned on its own: the compiler reads wsum[] with one 128-bit shared load, which
     // from an unaligned start also covered the last cur[] entry — racecheck reported that benign
     // over-read as a read/write hazard against the scan's cur[] stores
-    alignas(16) unsigned int wsum[kEmThreads / 32];
+    alignas(16) unsigned int wsum[kT / 32];
 };
 static_assert(kLsCapLarge <= 65536, "16-bit record ids");
 constexpr int kLcCapLarge = 8192;  // carry records per bucket in the large instance (~172 KB)
@@ -588,13 +588,16 @@ constexpr int kLcCapLarge = 8192;  // carry records per bucket in the large inst
 // bucket's first kPre * 256 records are loaded into registers while the current one is
 // decoded and stored, and its sub-bucket counters are cleared then too (one barrier less).
 constexpr int kPre = 3;
-template <int kCap, int kMin>
+// kT threads per block, at most kSub sub-buckets per bucket (a power of two).
+template <int kCap, int kMin, int kSub = kLsSubMax, int kT = kEmThreads>
 __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ kv,
                                                 const unsigned int *__restrict__ offset, int nb,
                                                 const Q18Plan *__restrict__ plan, const Q18Cols &dst,
                                                 unsigned int *flag, unsigned int *big, unsigned char *smem,
                                                 int sub_log2) {
-    LcSmem<kCap> &S = *reinterpret_cast<LcSmem<kCap> *>(smem);
+    LcSmem<kCap, kSub, kT> &S = *reinterpret_cast<LcSmem<kCap, kSub, kT> *>(smem);
+    constexpr int kQ = (kSub + kT - 1) / kT;  // sub-bucket counts scanned per thread
+    constexpr int kSubBits = kSub >= 4096 ? 12 : kSub >= 2048 ? 11 : kSub >= 1024 ? 10 : 9;
     const int shift = plan->shift;
     const Q18SortSpec sp = plan->spec;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -619,11 +622,11 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         }
 #pragma unroll
         for (int u = 0; u < kPre; ++u) {
-            const unsigned int i = threadIdx.x + u * kEmThreads;
+            const unsigned int i = threadIdx.x + u * kT;
             if (i < m) pre[u] = __ldcg(kv + lo + i);
         }
     };
-    for (unsigned int i = threadIdx.x; i <= kLsSubMax; i += kEmThreads) S.sub[i] = 0;
+    for (unsigned int i = threadIdx.x; i <= kSub; i += kT) S.sub[i] = 0;
     fetch(blockIdx.x);
     __syncthreads();
     for (int wi = blockIdx.x; wi < nwork; wi += gridDim.x) {
@@ -633,29 +636,29 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         }
         // sub-bucket bits: the smallest sb with (m >> (sb + sub_log2)) == 0, at most 10
         int sb = 32 - __clz(m) - sub_log2;
-        sb = sb < 0 ? 0 : sb > 9 ? 9 : sb;  // ns <= kLsSubMax
+        sb = sb < 0 ? 0 : sb > kSubBits ? kSubBits : sb;  // ns <= kSub
         if (sb > shift) sb = shift;
         const int ssh = shift - sb;
         const unsigned int ns = 1u << sb, smask = ns - 1u;
 #pragma unroll
         for (int u = 0; u < kPre; ++u) {
-            const unsigned int i = threadIdx.x + u * kEmThreads;
+            const unsigned int i = threadIdx.x + u * kT;
             if (i < m) {
                 S.rec[i] = pre[u];
                 atomicAdd(&S.sub[(unsigned int)(pre[u].x >> ssh) & smask], 1u);
             }
         }
-        for (unsigned int i = threadIdx.x + kPre * kEmThreads; i < m; i += kEmThreads) {  // rest
+        for (unsigned int i = threadIdx.x + kPre * kT; i < m; i += kT) {  // rest
             const ulonglong2 r = __ldcg(kv + lo + i);
             S.rec[i] = r;
             atomicAdd(&S.sub[(unsigned int)(r.x >> ssh) & smask], 1u);
         }
         __syncthreads();
-        {   // exclusive scan of ns (<= 1024) sub-bucket counts: 4 per thread
-            unsigned int c[4], t = 0;
+        {   // exclusive scan of ns (<= kSub) sub-bucket counts: kQ per thread
+            unsigned int c[kQ], t = 0;
 #pragma unroll
-            for (int q = 0; q < 4; ++q) {
-                const unsigned int i = threadIdx.x * 4 + q;
+            for (int q = 0; q < kQ; ++q) {
+                const unsigned int i = threadIdx.x * kQ + q;
                 c[q] = i < ns ? S.sub[i] : 0u;
                 t += c[q];
             }
@@ -671,21 +674,21 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
             for (int w = 0; w < warp; ++w) before += S.wsum[w];
             unsigned int run = before + x - t;
 #pragma unroll
-            for (int q = 0; q < 4; ++q) {
-                const unsigned int i = threadIdx.x * 4 + q;
+            for (int q = 0; q < kQ; ++q) {
+                const unsigned int i = threadIdx.x * kQ + q;
                 if (i < ns) { S.sub[i] = run; S.cur[i] = run; }
                 run += c[q];
             }
-            if (threadIdx.x == kEmThreads - 1) S.sub[ns] = run;
+            if (threadIdx.x == kT - 1) S.sub[ns] = run;
         }
         __syncthreads();
-        for (unsigned int i = threadIdx.x; i < m; i += kEmThreads) {
+        for (unsigned int i = threadIdx.x; i < m; i += kT) {
             const unsigned long long kk = S.rec[i].x;
             const unsigned int p = atomicAdd(&S.cur[(unsigned int)(kk >> ssh) & smask], 1u);
             S.idx[p] = (unsigned short)i;
         }
         __syncthreads();
-        for (unsigned int i = threadIdx.x; i < m; i += kEmThreads) {  // rank -> sorted order
+        for (unsigned int i = threadIdx.x; i < m; i += kT) {  // rank -> sorted order
             const unsigned int me = S.idx[i];
             const ulonglong2 r = S.rec[me];
             const unsigned int sbk = (unsigned int)(r.x >> ssh) & smask;
@@ -702,7 +705,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         __syncthreads();
         const unsigned int cur_lo = lo, cur_m = m;
         fetch(wi + gridDim.x);  // next bucket's records in flight during the stores below
-        for (unsigned int i = threadIdx.x; i <= ns; i += kEmThreads) S.sub[i] = 0;
+        for (unsigned int i = threadIdx.x; i <= ns; i += kT) S.sub[i] = 0;
         // decode + coalesced stores, two adjacent output rows per thread (8-byte stores of the
         // int32 columns, 16-byte of the int64 ones); an odd first / last row goes alone
         auto store1 = [&](unsigned int i) {
@@ -720,7 +723,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         };
         const unsigned int head = cur_lo & 1u;  // output row cur_lo + i is even for i = head
         const unsigned int npair = (cur_m - head) >> 1;
-        for (unsigned int p = threadIdx.x; p < npair; p += kEmThreads) {
+        for (unsigned int p = threadIdx.x; p < npair; p += kT) {
             const unsigned int i = head + 2 * p;
             const ulonglong2 ra = S.rec[S.srt[i]], rb = S.rec[S.srt[i + 1]];
             const CarryRow a = carry_decode(ra.x, ra.y, sp);
@@ -735,8 +738,8 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
             *reinterpret_cast<int2 *>(dst.o_w_id + j) = make_int2(a.o_w_id, b.o_w_id);
             *reinterpret_cast<int2 *>(dst.o_d_id + j) = make_int2(a.o_d_id, b.o_d_id);
         }
-        if (threadIdx.x == kEmThreads - 1 && head) store1(0);
-        if (threadIdx.x == kEmThreads - 2 && ((cur_m - head) & 1u)) store1(cur_m - 1);
+        if (threadIdx.x == kT - 1 && head) store1(0);
+        if (threadIdx.x == kT - 2 && ((cur_m - head) & 1u)) store1(cur_m - 1);
         __syncthreads();
     }
 }
@@ -935,6 +938,30 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
         }
         __syncthreads();
     }
+}
+
+// Buckets above the small instance's capacity, carry records only (v3 / distributed): 512 threads
+// and up to 4 096 sub-buckets per 8 192-record bucket in one 192 KB block per SM (the 128-thread
+// instance left 4 warps per SM for exactly the buckets that need the most work).
+constexpr int kLgThreads = 512;
+constexpr int kLgSub = 4096;
+constexpr size_t kLgSmem = sizeof(LcSmem<kLcCapLarge, kLgSub, kLgThreads>);
+__global__ void __launch_bounds__(kLgThreads, 1)
+carry_large_emit_kernel(const unsigned long long *__restrict__ k, const unsigned int *__restrict__ offset, int nb,
+                        const Q18Plan *__restrict__ plan, Q18Cols dst, unsigned int *flag, unsigned int *big,
+                        int sub_log2, PeerArgs pa) {
+    pdl_wait();
+    pdl_trigger();
+    extern __shared__ __align__(16) unsigned char smem_raw[];
+    if (pa.world > 1) {  // distributed ORDER BY: this rank's buckets in its heap (as the emit above)
+        const unsigned long long xs = plan->xseq;
+        if (plan->err & (kPeerErrHeap | kPeerErrOutCap | kPeerErrNoCarry | kPeerErrTimeout)) return;
+        k = reinterpret_cast<const unsigned long long *>(peer::heap(pa, pa.rank, (int)(xs & 1)));
+        nb = (int)plan->nb_mine;
+    }
+    if (!plan->spec.carry) return;
+    carry_sort_emit<kLcCapLarge, 1, kLgSub, kLgThreads>(reinterpret_cast<const ulonglong2 *>(k), offset, nb, plan,
+                                                      dst, flag, big, smem_raw, sub_log2);
 }
 
 // ============================================== bucket sort v2 (default) ===
@@ -1582,9 +1609,9 @@ void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, c
     count_launches(1);
     end();
     begin("q18_bucket_sort_emit_large");
-    launch_pdl(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>, (unsigned)num_sms, kEmThreads, kObSmemLarge, st,
-               (const unsigned long long *)bs.kv, (const unsigned int *)nullptr, (const unsigned int *)bs.offset, nb,
-               plan, (const Q18Row *)nullptr, (const long long *)nullptr, dst, flag, bs.big, sub_log2, PeerArgs{});
+    launch_pdl(carry_large_emit_kernel, (unsigned)num_sms, kLgThreads, kLgSmem, st,
+               (const unsigned long long *)bs.kv, (const unsigned int *)bs.offset, nb, plan, dst, flag, bs.big,
+               sub_log2, PeerArgs{});
     count_launches(1);
     end();
 }
@@ -1900,9 +1927,8 @@ void q18_dist_emit(const PeerArgs &pa, const Q18Plan *plan, const unsigned int *
     count_launches(1);
     end();
     begin("q18_bucket_sort_emit_large");
-    launch_pdl(bucket_local_emit_kernel<kLsCapLarge, kObCap, true>, (unsigned)num_sms, kEmThreads, kObSmemLarge, st,
-               (const unsigned long long *)nullptr, (const unsigned int *)nullptr, recv_off, 0, plan,
-               (const Q18Row *)nullptr, (const long long *)nullptr, dst, flag, s.big, sub_log2, pa);
+    launch_pdl(carry_large_emit_kernel, (unsigned)num_sms, kLgThreads, kLgSmem, st,
+               (const unsigned long long *)nullptr, recv_off, 0, plan, dst, flag, s.big, sub_log2, pa);
     count_launches(1);
     end();
 }
@@ -1945,7 +1971,8 @@ cudaError_t set_attributes_sort(int num_sms) {
         (const void *)q18_acc_stats_kernel,
         (const void *)q18_having_rec_kernel,
         (const void *)ob_scatter_rec_kernel,
-        (const void *)l2_touch_kernel};
+        (const void *)l2_touch_kernel,
+        (const void *)carry_large_emit_kernel};
     const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
     if (le != cudaSuccess) return le;
 
@@ -1962,6 +1989,7 @@ cudaError_t set_attributes_sort(int num_sms) {
         {(const void *)ob_scan_kernel, 4 * std::max(32 * G, 1 << kBucketMaxBits)},
         {(const void *)q18_dist_route_kernel, 4 << kBucketMaxBits},
         {(const void *)q18_having_rec_kernel, 4 << kBucketMaxBits},
+        {(const void *)carry_large_emit_kernel, (int)kLgSmem},
         {(const void *)ob_scatter_rec_kernel, 4 << kBucketMaxBits},
     };
     for (const auto &x : a) {
