@@ -1,10 +1,14 @@
 """World-size-2 CPU (gloo) coverage of the N>1 path's host logic: warehouse sharding and the
-merge semantics the library implements over NCCL:
+merge semantics the library implements:
   Q6  -> allreduce(sum) of {revenue, count}
   Q1  -> allgather of per-rank group lists, merge by key (integer sums)
-  Q18 -> gather of per-rank result rows to rank 0, re-sort by the ORDER BY key
+  Q18 -> groups are warehouse-local: the union of the shards' rows, ordered, is the whole result
+         (the library then range-partitions that order over the ranks)
 Each rank computes its partials with the oracle on its own shard; rank 0 checks the merged
-result against the oracle over all warehouses."""
+result against the oracle over all warehouses. This pins the DEFINITION of the merges (that they
+are exact under re-partitioning); the library's own world > 1 kernels run in
+tests/test_gpu_multirank.py (N logical ranks on one GPU, and two processes over CUDA IPC).
+bench.py's multi-rank launcher is checked here too (it refuses to run N ranks without N GPUs)."""
 import os
 import socket
 
@@ -54,7 +58,8 @@ def _worker(rank, world, port, q):
             for k, qty, amt, cnt in arr.tolist():
                 m = merged.setdefault(k, [0, 0, 0])
                 m[0] += qty; m[1] += amt; m[2] += cnt
-        # Q18: gather rows to rank 0
+        # Q18: groups are warehouse-local, so the union of the shards' result rows in the global
+        # ORDER BY is the whole result (the library range-partitions that order over the ranks)
         p18 = oracle.q18(part, Q18_HAVING)
         rows = list(zip(*[p18[n].tolist() for n, _ in oracle.Q18_COLUMNS]))
         gathered = [None] * world if rank == 0 else None
@@ -91,3 +96,21 @@ def test_gloo_sharded_merge_equals_whole(world):
         p.join(timeout=300)
         assert p.exitcode == 0
     assert q.get(timeout=10) is True
+
+
+def test_bench_refuses_more_ranks_than_gpus():
+    """bench.py --gpus 2 without a torchrun environment spawns its ranks itself only when two
+    GPUs are visible; otherwise it reports the error and exits non-zero (never a silent N=1)."""
+    import subprocess
+    import sys
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    env = {k: v for k, v in os.environ.items() if k not in ("RANK", "WORLD_SIZE", "LOCAL_RANK")}
+    env["CUDA_VISIBLE_DEVICES"] = ""
+    r = subprocess.run([sys.executable, os.path.join(root, "bench.py"), "--gpus", "2", "--steps", "1"],
+                       capture_output=True, text=True, env=env, timeout=600)
+    assert r.returncode != 0
+    assert "error" in r.stdout and "--gpus 2" in r.stdout
+    env.update(RANK="0", WORLD_SIZE="1", LOCAL_RANK="0")
+    r = subprocess.run([sys.executable, os.path.join(root, "bench.py"), "--gpus", "2", "--steps", "1"],
+                       capture_output=True, text=True, env=env, timeout=600)
+    assert r.returncode != 0 and "WORLD_SIZE=1" in r.stdout
