@@ -68,17 +68,33 @@ __global__ void q18_build_kernel(const int32_t *__restrict__ o_w, const int32_t 
                                  const int32_t *__restrict__ c_id, uint64_t n_c, Q18Scratch s) {
     pdl_wait();
     pdl_trigger();
+    // U rows per thread per iteration: their key loads, then their inserts (atomicCAS with
+    // return: a dependent round trip) are independent, so U of each are in flight per thread
+    // (one row per iteration left the kernel waiting on one CAS at a time: 39 us)
+    constexpr int U = 4;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n_o + n_c; i += stride) {
-        bool ok;
-        if (i < n_o) {
-            reinterpret_cast<ulonglong2 *>(s.acc)[i] = make_ulonglong2(0ull, 0ull);  // acc[orders row]
-            ok = jx_insert(s.jo, o_w[i], o_d[i], o_id[i], (unsigned int)i, s.err, kErrDupOrders);
-        } else {
-            const uint64_t j = i - n_o;
-            ok = jx_insert(s.jc, c_w[j], c_d[j], c_id[j], (unsigned int)j, s.err, kErrDupCustomer);
+    const uint64_t total = n_o + n_c;
+    for (uint64_t i0 = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i0 < total; i0 += U * stride) {
+        int w[U], d[U], k[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const uint64_t i = i0 + u * stride;
+            if (i < n_o) { w[u] = __ldcs(o_w + i); d[u] = __ldcs(o_d + i); k[u] = __ldcs(o_id + i); }
+            else if (i < total) { const uint64_t j = i - n_o; w[u] = __ldcs(c_w + j); d[u] = __ldcs(c_d + j); k[u] = __ldcs(c_id + j); }
         }
-        if (!ok) atomicOr(s.err, kErrDomain);
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const uint64_t i = i0 + u * stride;
+            if (i >= total) break;
+            bool ok;
+            if (i < n_o) {
+                reinterpret_cast<ulonglong2 *>(s.acc)[i] = make_ulonglong2(0ull, 0ull);  // acc[orders row]
+                ok = jx_insert(s.jo, w[u], d[u], k[u], (unsigned int)i, s.err, kErrDupOrders);
+            } else {
+                ok = jx_insert(s.jc, w[u], d[u], k[u], (unsigned int)(i - n_o), s.err, kErrDupCustomer);
+            }
+            if (!ok) atomicOr(s.err, kErrDomain);
+        }
     }
 }
 
@@ -516,7 +532,7 @@ void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaSt
 void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
                       const int32_t *c_w, const int32_t *c_d, const int32_t *c_id, uint64_t n_c,
                       const Q18Scratch &s, int num_sms, cudaStream_t st) {
-    launch_pdl(q18_build_kernel, grid_for(n_o + n_c, 256, num_sms, 8), 256, 0, st, o_w, o_d, o_id, n_o, c_w,
+    launch_pdl(q18_build_kernel, grid_for((n_o + n_c + 3) / 4, 256, num_sms, 8), 256, 0, st, o_w, o_d, o_id, n_o, c_w,
                                                                          c_d, c_id, n_c, s);
     count_launches(1);
 }

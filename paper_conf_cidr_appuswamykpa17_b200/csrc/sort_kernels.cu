@@ -1343,7 +1343,7 @@ q18_acc_stats_kernel(const Q18Acc *__restrict__ acc, const int64_t *__restrict__
     long long amin = INT64_MAX, amax = INT64_MIN, emin = INT64_MAX, emax = INT64_MIN;
     unsigned long long c = 0;
     const uint64_t stride = (uint64_t)gridDim.x * kStatThreads;
-    constexpr int U = 4;  // independent accumulator loads in flight per thread
+    constexpr int U = 8;  // independent accumulator loads in flight per thread
     for (uint64_t r0 = (uint64_t)blockIdx.x * kStatThreads + threadIdx.x; r0 < n_o; r0 += U * stride) {
         ulonglong2 a[U];
 #pragma unroll
@@ -1554,7 +1554,7 @@ void launch_q18_acc_stats(const Q18Scratch &s, const int64_t *o_ent, uint64_t n_
                           unsigned long long *cpart, unsigned long long *count, const Q18PlanArgs *plan_args,
                           int bucket_bits, Q18Plan *plan, unsigned int *flag, int num_sms, cudaStream_t st) {
     uint64_t want = (n_o + kStatThreads - 1) / kStatThreads;
-    const uint64_t cap = (uint64_t)num_sms * 8;  // = the stat_part capacity (8 blocks per SM)
+    const uint64_t cap = (uint64_t)num_sms * 4;  // <= the stat_part capacity (8 blocks per SM)
     const unsigned grid = (unsigned)(want < 1 ? 1 : want > cap ? cap : want);
     const Q18Zone z = plan_args ? plan_args->zone : Q18Zone{};
     launch_pdl(q18_acc_stats_kernel, grid, kStatThreads, 0, st, (const Q18Acc *)s.acc, o_ent, n_o,
