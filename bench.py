@@ -58,6 +58,8 @@ def parse():
                     help="strong scaling: this many warehouses split over the GPUs (config C4)")
     ap.add_argument("--peer-heap-mb", type=int, default=0, help="world > 1: peer heap per rank (0 = 1 GiB)")
     ap.add_argument("--no-c1", action="store_true", help="skip the config C1 line (Q6 at W=1)")
+    ap.add_argument("--sleep-cycles", type=int, default=200_000,
+                    help="sleep kernel queued before each timed step (the host enqueues meanwhile)")
     ap.add_argument("--plans", default="q6,q1,q18",
                     help="the step's queries (config C4 is Q1 + Q6: --plans q6,q1)")
     ap.add_argument("--mode", default="spread", choices=["spread", "strict"])
@@ -440,8 +442,10 @@ def main():
     plans = tuple(p for p in (("q6", h.H2TAP_Q6, Q6_P), ("q1", h.H2TAP_Q1, Q1_P), ("q18", h.H2TAP_Q18, Q18_P))
                   if p[0] in want)
 
-    def run_batch(sel, flags):
+    def run_batch(sel, flags, end_event=None):
         rs = h.h2tap_run_queries(eng, [(plan, p, flags) for name, plan, p in plans if name in sel])
+        if end_event is not None:  # right after the call returns (the batch is complete on the
+            end_event.record(stream)  # device): the Python bookkeeping below stays outside
         out = {}
         for name, r in zip([n for n, _, _ in plans if n in sel], rs):
             out[name] = (r.device_ms, r.kernels if flags & h.H2TAP_QUERY_PROFILE else [], r.nrows,
@@ -477,10 +481,9 @@ def main():
     for i in range(a.steps):
         flush_l2()
         with torch.cuda.stream(stream):  # ~50 us sleep outside the events: the host enqueues the
-            torch.cuda._sleep(200_000)   # batch while the GPU sleeps (no launch gap inside)
+            torch.cuda._sleep(a.sleep_cycles)  # batch while the GPU sleeps (no launch gap inside)
         starts[i].record(stream)
-        out = run_batch(ALL, dev_flags)
-        ends[i].record(stream)
+        out = run_batch(ALL, dev_flags, ends[i])
         for q, (ms, ks, nrows, nl, tot) in out.items():
             per_query[q].append(ms)
             launches += nl
@@ -502,7 +505,7 @@ def main():
         for _ in range(a.steps):
             flush_l2()
             with torch.cuda.stream(stream):
-                torch.cuda._sleep(200_000)
+                torch.cuda._sleep(a.sleep_cycles)
             ms.append(run_batch((q,), dev_flags)[q][0])
         alone[q] = float(np.median(ms))
     barrier()
