@@ -1849,6 +1849,10 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
     // with per-kernel profiling, a short gate lets the whole batch be enqueued before the GPU
     // starts it, so no kernel's event window contains host launch latency
     if (profile) launch_gate(30000, e->compute);
+    // with world > 1, profiling also aligns the ranks first (a data-less collective): the per-kernel
+    // windows then hold each merge's own cost, not the host-side skew between the ranks' launches
+    if (profile && e->world > 1)
+        launch_peer_allreduce_i64(e->peer.args, nullptr, 0, nullptr, nullptr, e->compute);
     struct Cleanup {  // return pooled blocks of queries that did not complete
         h2tap_engine *e; std::vector<QueryCtx> &c;
         ~Cleanup() {

@@ -92,10 +92,13 @@ void launch_peer_allreduce_i64(const PeerArgs &p, const long long *src, int n, l
 
 void launch_peer_push(const PeerArgs &p, const void *src, const unsigned long long *count_dev,
                       unsigned long long count_const, unsigned int elem_bytes, int num_sms, cudaStream_t st) {
-    // enough blocks for ~2 MB lists at 16 B per thread; a handful suffices for the typical KBs
+    // the lists are small (Q1: <= 16 groups on TPC-C data; ORDER BY counts: <= 128 KB) and every
+    // block ends with a system-scope fence before the last-block ticket: a few blocks, each
+    // looping, instead of a block per SM (a 2 MB worst-case list then takes ~16 iterations)
     const unsigned long long max_bytes = count_dev ? p.slot_bytes - 16 : count_const * elem_bytes;
     unsigned long long blocks = (max_bytes / 16 + 255) / 256;
-    if (blocks > (unsigned long long)num_sms) blocks = (unsigned long long)num_sms;
+    const unsigned long long cap = (unsigned long long)(num_sms < 32 ? num_sms : 32);
+    if (blocks > cap) blocks = cap;
     if (blocks < 1) blocks = 1;
     launch_pdl(peer_push_kernel, (unsigned)blocks, 256, 0, st, p, src, count_dev, count_const, elem_bytes);
     count_launches(1);
