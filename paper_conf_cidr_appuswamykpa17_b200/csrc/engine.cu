@@ -391,6 +391,7 @@ struct h2tap_engine {
     // kernels can overlap the bandwidth-bound scans of the other queries
     cudaStream_t side = nullptr;
     bool q18_side = false;
+    bool q1_side = true;   // H2TAP_Q1_SIDE=0: a shared-scan Q1's compact + emit stay on the compute stream
     cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
     cudaStream_t reaper = nullptr;  // stream-ordered frees of snapshot buffers
     FreeOrder free_order;
@@ -1915,9 +1916,20 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
         q.mark0 = e->prof.marks.size();
         q.launches0 = launches_total();
         // Q18 / Q3 on the side stream (only when something else in the batch could overlap)
-        const bool on_side = e->q18_side && n > 1 && (q.plan == H2TAP_Q18 || q.plan == H2TAP_Q3);
-        if (on_side && !forked) {  // fork from the batch start: the side work need not wait for
-                                   // the queries enqueued before it on the compute stream
+        // The tail of a Q1 whose scan ran in the batch's shared pass (compact + emit, two small
+        // latency-bound kernels) goes to the side stream, forked right after that pass, when more
+        // queries follow: it overlaps the next query's first kernels instead of delaying them
+        // (one GPU only: with world > 1 every collective must stay in one stream order, the same
+        // on every rank, because their sequence numbers come from one device counter)
+        const bool q1_tail = e->q1_side && e->world == 1 && q.plan == H2TAP_Q1 && q.shared_scan == 2 &&
+                             i + 1 < ctx.size() && !forked;
+        const bool on_side = q1_tail || (e->q18_side && n > 1 && (q.plan == H2TAP_Q18 || q.plan == H2TAP_Q3));
+        if (q1_tail) {  // fork point: now (the compute stream's last work is the shared scan)
+            CK(cudaEventRecord(e->ev_fork, e->compute));
+            CK(cudaStreamWaitEvent(e->side, e->ev_fork, 0));
+            forked = true;
+        } else if (on_side && !forked) {  // fork from the batch start: the side work need not
+                                          // wait for the queries enqueued before it
             CK(cudaStreamWaitEvent(e->side, e->ev_fork, 0));
             forked = true;
         }
@@ -2041,6 +2053,7 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         CK(cudaEventCreateWithFlags(&e->ev_fork, cudaEventDisableTiming));
         CK(cudaEventCreateWithFlags(&e->ev_join, cudaEventDisableTiming));
         if (const char *q = std::getenv("H2TAP_Q18_STREAM")) e->q18_side = std::atoi(q) != 0;
+        if (const char *q = std::getenv("H2TAP_Q1_SIDE")) e->q1_side = std::atoi(q) != 0;
         CK(cudaStreamCreateWithFlags(&e->reaper, cudaStreamNonBlocking));
         e->free_order = FreeOrder{e->compute, e->copy, e->reaper};
         {   // keep freed pool memory cached (no release to the OS at stream syncs)
