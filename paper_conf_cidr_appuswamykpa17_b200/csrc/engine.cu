@@ -1849,7 +1849,11 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
     e->prof.reset(profile, e->compute);
     // with per-kernel profiling, a short gate lets the whole batch be enqueued before the GPU
     // starts it, so no kernel's event window contains host launch latency
-    if (profile) launch_gate(30000, e->compute);
+    static const unsigned long long gate_ns = [] {  // H2TAP_PROFILE_GATE_US (default 30)
+        const char *v = std::getenv("H2TAP_PROFILE_GATE_US");
+        return (unsigned long long)((v ? std::atof(v) : 30.0) * 1000.0);
+    }();
+    if (profile) launch_gate(gate_ns, e->compute);
     // with world > 1, profiling also aligns the ranks first (a data-less collective): the per-kernel
     // windows then hold each merge's own cost, not the host-side skew between the ranks' launches
     if (profile && e->world > 1)
