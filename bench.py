@@ -58,6 +58,9 @@ def parse():
                     help="strong scaling: this many warehouses split over the GPUs (config C4)")
     ap.add_argument("--peer-heap-mb", type=int, default=0, help="world > 1: peer heap per rank (0 = 1 GiB)")
     ap.add_argument("--no-c1", action="store_true", help="skip the config C1 line (Q6 at W=1)")
+    ap.add_argument("--share-device", action="store_true",
+                    help="functional check of the N-rank path on ONE GPU: every rank on cuda:0 (CUDA IPC between "
+                         "the processes), gloo for the plumbing; timings meaningless, never a bench line")
     ap.add_argument("--sleep-cycles", type=int, default=200_000,
                     help="sleep kernel queued before each timed step (the host enqueues meanwhile)")
     ap.add_argument("--plans", default="q6,q1,q18",
@@ -82,7 +85,7 @@ def spawn_ranks(a):
     import socket
     import torch
     have = torch.cuda.device_count()
-    if have < a.gpus:
+    if have < a.gpus and not (a.share_device and have >= 1):
         print(json.dumps({"error": f"--gpus {a.gpus} but {have} CUDA device(s) visible"}), flush=True)
         return 2
     s = socket.socket()
@@ -395,9 +398,15 @@ def main():
     import torch
     import torch.distributed as dist
 
+    if a.share_device:
+        local = 0
     torch.cuda.set_device(local)
+    pg_dev = "cpu" if a.share_device else "cuda"  # gloo reduces host tensors, NCCL device tensors
     if world > 1:  # plumbing only: peer-handle exchange, barriers, max-over-ranks timing
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        if a.share_device:
+            dist.init_process_group("gloo")
+        else:
+            dist.init_process_group("nccl", device_id=torch.device("cuda", local))
 
     import paper_conf_cidr_appuswamykpa17_b200 as h
 
@@ -433,7 +442,7 @@ def main():
         torch.cuda.synchronize()
 
     def max_over_ranks(vals):
-        t = torch.tensor(vals, dtype=torch.float64, device="cuda")
+        t = torch.tensor(vals, dtype=torch.float64, device=pg_dev)
         if world > 1:
             dist.all_reduce(t, op=dist.ReduceOp.MAX)
         return [float(x) for x in t.tolist()]
@@ -525,7 +534,7 @@ def main():
                                                        alone.get("q1", float("nan"))])
     lat = {q: float(np.median(v)) for q, v in per_query.items()}
     lat_max = dict(zip(lat, max_over_ranks(list(lat.values()))))
-    nt = torch.tensor([n_ol], dtype=torch.float64, device="cuda")
+    nt = torch.tensor([n_ol], dtype=torch.float64, device=pg_dev)
     if world > 1:
         dist.all_reduce(nt, op=dist.ReduceOp.SUM)
     rows_total = int(nt.item())  # order_line rows of all ranks, each counted once per step
@@ -636,7 +645,8 @@ def main():
                        "orders_rows_rank0": n_o, "customer_rows_rank0": n_c,
                        "rows_counted": ("each visible order_line row counted once per step; one step = CH "
                                         + " + ".join(q.upper() for q in ALL) + " over the snapshot"),
-                       "queries_per_step": len(ALL), "parallelism": f"row-sharded by warehouse x{world}",
+                       "queries_per_step": len(ALL),
+                       **({"shared_device": "FUNCTIONAL CHECK ONLY: all ranks on one GPU"} if a.share_device else {}), "parallelism": f"row-sharded by warehouse x{world}",
                        "merge": ("peer-memory kernels over NVLink (Q6 allreduce, Q1 group lists, Q18 "
                                  "range-partitioned ORDER BY; DESIGN.md §6)" if world > 1 else "none (1 GPU)"),
                        "scan_sharing": ("Q6 and Q1 of the batch share one pass over order_line "

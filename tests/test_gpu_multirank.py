@@ -300,3 +300,21 @@ def test_two_processes_one_gpu_ipc(h, tmp_path):
     for r, p in enumerate(procs):
         assert p.returncode == 0, f"rank {r}:\n{outs[r][-3000:]}"
         assert "RANK_OK" in outs[r], outs[r][-2000:]
+
+
+def test_bench_two_ranks_functional():
+    """bench.py's N-rank path end to end (it spawns its ranks, maps the peer segments over the
+    process group, takes the max over ranks, sums the rows): --share-device puts both ranks on the
+    one GPU (CUDA IPC between processes, gloo plumbing). Functional only: the line says so."""
+    import json as _json
+    env = {k: v for k, v in os.environ.items() if k not in ("RANK", "WORLD_SIZE", "LOCAL_RANK")}
+    r = subprocess.run([sys.executable, os.path.join(ROOT, "bench.py"), "--gpus", "2", "--share-device",
+                        "--steps", "2", "--warmup", "3", "--warehouses", "2", "--no-cpu-baseline", "--no-c1",
+                        "--e2e-steps", "2"], capture_output=True, text=True, env=env, timeout=600)
+    assert r.returncode == 0, r.stderr[-3000:]
+    line = _json.loads([x for x in r.stdout.splitlines() if x.startswith("{")][-1])
+    assert line["n_gpus"] == 2 and line["config"]["shared_device"]
+    whole = chgen.generate(1, 5, seed=1)
+    assert line["config"]["order_line_rows_total"] == len(whole["order_line"]["ol_w_id"])
+    assert line["q18_result_rows_total"] == len(oracle.q18(whole, Q18_HAVING)["o_id"])
+    assert line["gpu_launches"] > 0 and line["value"] > 0
