@@ -391,6 +391,7 @@ struct h2tap_engine {
     // kernels can overlap the bandwidth-bound scans of the other queries
     cudaStream_t side = nullptr;
     bool q18_side = false;
+    uint64_t q18_runs = 0;  // Q18 / Q3 launches: parity of the clustered-index counters
     bool q1_side = true;   // H2TAP_Q1_SIDE=0: a shared-scan Q1's compact + emit stay on the compute stream
     cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
     cudaStream_t reaper = nullptr;  // stream-ordered frees of snapshot buffers
@@ -1218,6 +1219,16 @@ void q18_scratch(h2tap_engine *e, const View &v, QueryCtx &q, uint64_t rows_cap)
     Q18Scratch &s = q.q18;
     s.jo = plan_index(e, v, O, force_hash, "q18.jo");
     s.jc = plan_index(e, v, C, force_hash, "q18.jc");
+    {   // clustered build sides (row == dense slot), verified on the device by the init kernel;
+        // counters per query parity (the init of query k clears those of query k+1)
+        auto *viol = static_cast<unsigned int *>(e->arena.get("q18.viol", 64, true, e->compute));
+        const int par = (int)(e->q18_runs++ & 1);
+        static const bool on = [] { const char *x = std::getenv("H2TAP_CLUSTERED"); return !(x && x[0] == '0'); }();
+        s.jo.may_ident = on && s.jo.dense && s.jo.range == v.n[O];
+        s.jc.may_ident = on && s.jc.dense && s.jc.range == v.n[C];
+        s.jo.viol = viol + 2 * par; s.jo.viol_next = viol + 2 * (par ^ 1);
+        s.jc.viol = viol + 2 * par + 1; s.jc.viol_next = viol + 2 * (par ^ 1) + 1;
+    }
     s.acc = static_cast<Q18Acc *>(e->arena.get("q18.acc", sizeof(Q18Acc) * std::max<uint64_t>(n_o, 1)));
     s.err = static_cast<unsigned int *>(e->arena.get("q18.err", 64));
     s.nout = static_cast<unsigned long long *>(e->arena.get("q18.nout", 64));
@@ -1352,7 +1363,12 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     q18_scratch(e, v, q, n_o);
     Q18Scratch &s = q.q18;
 
-    e->prof.run("q18_init", [&] { launch_q18_init(s, n_o, e->num_sms, e->compute); });
+    e->prof.run("q18_init", [&] {
+        launch_q18_init(s, colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
+                        colp<int32_t>(v, O, H2TAP_O_ID), n_o, colp<int32_t>(v, C, H2TAP_C_W_ID),
+                        colp<int32_t>(v, C, H2TAP_C_D_ID), colp<int32_t>(v, C, H2TAP_C_ID), n_c, e->num_sms,
+                        e->compute);
+    });
     e->prof.run("q18_build", [&] {
         launch_q18_build(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
                          colp<int32_t>(v, O, H2TAP_O_ID), n_o, colp<int32_t>(v, C, H2TAP_C_W_ID),
@@ -1442,7 +1458,12 @@ void launch_q3_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     s.ncand = static_cast<unsigned long long *>(e->arena.get("q3.ncand", 64));
     s.qwords = (n_o + 31) / 32;
     s.qbits = static_cast<unsigned int *>(e->arena.get("q3.bits", 4 * std::max<uint64_t>(s.qwords, 1)));
-    e->prof.run("q3_init", [&] { launch_q18_init(s, n_o, e->num_sms, e->compute); });
+    e->prof.run("q3_init", [&] {
+        launch_q18_init(s, colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
+                        colp<int32_t>(v, O, H2TAP_O_ID), n_o, colp<int32_t>(v, C, H2TAP_C_W_ID),
+                        colp<int32_t>(v, C, H2TAP_C_D_ID), colp<int32_t>(v, C, H2TAP_C_ID), n_c, e->num_sms,
+                        e->compute);
+    });
     e->prof.run("q3_build", [&] {
         launch_q18_build(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
                          colp<int32_t>(v, O, H2TAP_O_ID), n_o, colp<int32_t>(v, C, H2TAP_C_W_ID),

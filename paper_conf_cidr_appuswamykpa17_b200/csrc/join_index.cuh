@@ -49,10 +49,16 @@ __device__ __forceinline__ bool jx_insert(const JoinIndex &j, int w, int d, int 
     }
 }
 
+// The build side is stored in key order with no gap (verified by the init kernel): row == slot.
+__device__ __forceinline__ bool jx_identity(const JoinIndex &j) {
+    return j.dense && j.may_ident && __ldg(j.viol) == 0u;
+}
+
 __device__ __forceinline__ unsigned int jx_lookup(const JoinIndex &j, int w, int d, int id) {
     if (j.dense) {
         unsigned long long s;
         if (!dense_slot(j, w, d, id, s)) return kNoRow;  // outside the build box: no match
+        if (jx_identity(j)) return (unsigned int)s;       // clustered build side: positional
         return __ldcg(j.slots + s);
     }
     unsigned long long key;

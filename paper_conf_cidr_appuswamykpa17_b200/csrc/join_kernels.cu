@@ -39,10 +39,54 @@ unsigned grid_for(uint64_t work, int threads, int num_sms, int per_sm) {
 // ------------------------------------------------------------------- init --
 // Empties both join indexes, zeroes the group accumulators and the counters: one launch.
 // Empties both join indexes, zeroes the group accumulators and the counters: one launch.
+// Does every build row sit at its own dense slot (row == rank of its key in the box)? Counts the
+// rows that do not (a warp-aggregated atomic per warp with any): 0 = the index is the identity.
+__device__ __forceinline__ void verify_identity(const JoinIndex &j, const int32_t *w, const int32_t *d,
+                                                const int32_t *id, uint64_t n, Q18Acc *acc = nullptr) {
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    const uint64_t n_pad = (n + 31) & ~31ull;  // whole warps (ballot)
+    constexpr int U = 4;                       // independent key loads in flight per thread
+    for (uint64_t r0 = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; r0 < n_pad; r0 += U * stride) {
+        int kw[U], kd[U], ki[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const uint64_t r = r0 + u * stride;
+            if (r < n) { kw[u] = __ldcs(w + r); kd[u] = __ldcs(d + r); ki[u] = __ldcs(id + r); }
+        }
+        unsigned int bad = 0;
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const uint64_t r = r0 + u * stride;
+            unsigned long long s;
+            bad += r < n && (!dense_slot(j, kw[u], kd[u], ki[u], s) || s != r);
+            if (acc && r < n) reinterpret_cast<ulonglong2 *>(acc)[r] = make_ulonglong2(0ull, 0ull);
+        }
+        const unsigned int b = __ballot_sync(__activemask(), bad != 0);
+        if (b && (threadIdx.x & 31) == __ffs(b) - 1) atomicAdd(j.viol, 1u);  // (a count > 0 suffices)
+    }
+}
+
+// Clustered build sides: count the rows not at their own dense slot; reset the
+// counters of the next query. Runs before the init, which then need not clear an identity index.
+__global__ void q18_verify_kernel(Q18Scratch s, const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
+                                  const int32_t *__restrict__ o_id, uint64_t n_o, const int32_t *__restrict__ c_w,
+                                  const int32_t *__restrict__ c_d, const int32_t *__restrict__ c_id, uint64_t n_c) {
+    pdl_wait();
+    pdl_trigger();
+    if (s.jo.may_ident) verify_identity(s.jo, o_w, o_d, o_id, n_o, s.acc);  // (+ zeroes acc: no build pass)
+    if (s.jc.may_ident) verify_identity(s.jc, c_w, c_d, c_id, n_c);
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
+        if (s.jo.viol_next) *s.jo.viol_next = 0u;
+        if (s.jc.viol_next) *s.jc.viol_next = 0u;
+    }
+}
+
 __global__ void q18_init_kernel(Q18Scratch s) {
     pdl_wait();
     pdl_trigger();
-    const uint64_t a = jx_words(s.jo), b = jx_words(s.jc), q = s.qbits ? s.qwords : 0;
+    // an identity index is never read: nothing to clear (the verify kernel ran before)
+    const uint64_t a = jx_identity(s.jo) ? 0 : jx_words(s.jo), b = jx_identity(s.jc) ? 0 : jx_words(s.jc);
+    const uint64_t q = s.qbits ? s.qwords : 0;
     const uint64_t total = a + b + q;  // (the accumulators are zeroed by the build, row by row)
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < total; i += stride) {
@@ -74,23 +118,26 @@ __global__ void q18_build_kernel(const int32_t *__restrict__ o_w, const int32_t 
     constexpr int U = 4;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     const uint64_t total = n_o + n_c;
+    const bool ident_o = jx_identity(s.jo), ident_c = jx_identity(s.jc);  // positional: no insert
+    if (ident_o && ident_c && s.jo.may_ident) return;  // nothing to insert, acc zeroed by the verify
     for (uint64_t i0 = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i0 < total; i0 += U * stride) {
         int w[U], d[U], k[U];
 #pragma unroll
-        for (int u = 0; u < U; ++u) {
+        for (int u = 0; u < U; ++u) {  // (an identity side needs no keys: nothing is inserted)
             const uint64_t i = i0 + u * stride;
-            if (i < n_o) { w[u] = __ldcs(o_w + i); d[u] = __ldcs(o_d + i); k[u] = __ldcs(o_id + i); }
-            else if (i < total) { const uint64_t j = i - n_o; w[u] = __ldcs(c_w + j); d[u] = __ldcs(c_d + j); k[u] = __ldcs(c_id + j); }
+            if (i < n_o) { if (!ident_o) { w[u] = __ldcs(o_w + i); d[u] = __ldcs(o_d + i); k[u] = __ldcs(o_id + i); } }
+            else if (i < total && !ident_c) { const uint64_t j = i - n_o; w[u] = __ldcs(c_w + j); d[u] = __ldcs(c_d + j); k[u] = __ldcs(c_id + j); }
         }
 #pragma unroll
         for (int u = 0; u < U; ++u) {
             const uint64_t i = i0 + u * stride;
             if (i >= total) break;
-            bool ok;
+            bool ok = true;
             if (i < n_o) {
-                reinterpret_cast<ulonglong2 *>(s.acc)[i] = make_ulonglong2(0ull, 0ull);  // acc[orders row]
-                ok = jx_insert(s.jo, w[u], d[u], k[u], (unsigned int)i, s.err, kErrDupOrders);
-            } else {
+                if (!s.jo.may_ident)  // (else the verify kernel zeroed it)
+                    reinterpret_cast<ulonglong2 *>(s.acc)[i] = make_ulonglong2(0ull, 0ull);  // acc[orders row]
+                if (!ident_o) ok = jx_insert(s.jo, w[u], d[u], k[u], (unsigned int)i, s.err, kErrDupOrders);
+            } else if (!ident_c) {
                 ok = jx_insert(s.jc, w[u], d[u], k[u], (unsigned int)(i - n_o), s.err, kErrDupCustomer);
             }
             if (!ok) atomicOr(s.err, kErrDomain);
@@ -522,8 +569,14 @@ void launch_q18_publish(const unsigned long long *nout, const unsigned int *err,
     count_launches(1);
 }
 
-void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st) {
-    (void)n_orders;
+void launch_q18_init(const Q18Scratch &s, const int32_t *o_w, const int32_t *o_d, const int32_t *o_id,
+                     uint64_t n_o, const int32_t *c_w, const int32_t *c_d, const int32_t *c_id, uint64_t n_c,
+                     int num_sms, cudaStream_t st) {
+    if (s.jo.may_ident || s.jc.may_ident) {
+        launch_pdl(q18_verify_kernel, grid_for((n_o + n_c + 3) / 4, 256, num_sms, 8), 256, 0, st,
+                   s, o_w, o_d, o_id, n_o, c_w, c_d, c_id, n_c);
+        count_launches(1);
+    }
     const uint64_t words = jx_words(s.jo) + jx_words(s.jc);
     launch_pdl(q18_init_kernel, grid_for(words, 256, num_sms, 8), 256, 0, st, s);
     count_launches(1);
@@ -618,6 +671,7 @@ cudaError_t set_attributes_join(int num_sms) {
         (const void *)q18_having_kernel<2>,
         (const void *)q18_having_kernel<4>,
         (const void *)q18_init_kernel,
+        (const void *)q18_verify_kernel,
         (const void *)q18_probe_kernel<false>,
         (const void *)q18_probe_kernel<true>,
         (const void *)q18_probe_tma_kernel,

@@ -124,6 +124,13 @@ struct JoinIndex {
     int w0, d0, k0;                                   // dense: box minimum
     unsigned int nw, nd, nk;                          // dense: box extents
     unsigned long long range;                         // dense: nw * nd * nk
+    // dense and exactly one build row per box slot (n == range): the build side MAY be stored in
+    // key order ("clustered"), i.e. row == slot for every row. The init kernel verifies that,
+    // counting violations into *viol; while *viol == 0 lookups return the slot itself (no slot
+    // read, no insert at build: DESIGN.md §4.3). A counter per index per query parity; the init of
+    // query k clears the counters query k+1 uses.
+    int may_ident;
+    unsigned int *viol, *viol_next;
 };
 struct Q18Stats {            // min/max of the sort fields that only the result rows know
     long long amt_min, amt_max, ent_min, ent_max;
@@ -158,7 +165,10 @@ struct Q18Scratch {
     unsigned long long qwords;
     unsigned int *tie;       // ORDER BY flag word, zeroed by init (null: not zeroed)
 };
-void launch_q18_init(const Q18Scratch &s, uint64_t n_orders, int num_sms, cudaStream_t st);
+// empties both join indexes (and verifies a clustered build side: JoinIndex::may_ident)
+void launch_q18_init(const Q18Scratch &s, const int32_t *o_w, const int32_t *o_d, const int32_t *o_id,
+                     uint64_t n_o, const int32_t *c_w, const int32_t *c_d, const int32_t *c_id, uint64_t n_c,
+                     int num_sms, cudaStream_t st);
 void launch_q18_build(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
                       const int32_t *c_w, const int32_t *c_d, const int32_t *c_id, uint64_t n_c,
                       const Q18Scratch &s, int num_sms, cudaStream_t st);
