@@ -695,3 +695,35 @@ def test_full_size_w1000_q6_q1_shared_batch(h):
         assert_q1(L.q(1), want1)
     finally:
         h.h2tap_close(e)
+
+
+@pytest.mark.parametrize("layout", ["clustered", "one_row_swapped", "shuffled", "customer_shuffled"])
+def test_q18_clustered_index_verification(L, layout, order_mode):
+    """The positional (clustered) join index is used only while the device finds
+    every build row at its own key slot: a generated table (in key order), one swapped pair of
+    orders rows, fully shuffled orders, shuffled customers — all must equal the oracle, on the
+    perfect-hash and the hash-join plans, Q18 and Q3."""
+    from test_oracle_q3 import Q3_LO
+    t = chgen.generate(1, 3, seed=41)
+    rng = np.random.default_rng(41)
+    o, c = t["orders"], t["customer"]
+    if layout == "one_row_swapped":
+        perm = np.arange(len(o["o_id"]))
+        perm[[10, 20000]] = perm[[20000, 10]]
+        t["orders"] = {k: v[perm].copy() for k, v in o.items()}
+    elif layout == "shuffled":
+        perm = rng.permutation(len(o["o_id"]))
+        t["orders"] = {k: v[perm].copy() for k, v in o.items()}
+    elif layout == "customer_shuffled":
+        perm = rng.permutation(len(c["c_id"]))
+        t["customer"] = {k: v[perm].copy() for k, v in c.items()}
+    L.h.h2tap_load_snapshot(L.e, L.h.hot_path_tables(t, (L.h.H2TAP_Q18, L.h.H2TAP_Q3)), L.epoch + 1)
+    L.epoch += 1
+    for thr in (Q18_HAVING, 4_000_000):
+        want = oracle.q18(t, thr)
+        assert_q18(L.q(18, [thr]), want)
+        assert_q18(L.q(18, [thr], flags=HASH), want)
+    want3 = oracle.q3(t, Q3_LO, b"A")
+    got3 = L.q(3, [Q3_LO, 0x4100])
+    for k in want3:
+        assert np.array_equal(got3[k], want3[k]), k
