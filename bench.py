@@ -198,10 +198,20 @@ def key_box(t, cols):
     return n
 
 
-def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None):
+def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None, clustered=False):
     """Bytes the method must move per launch. `box`: the
     (orders, customer) key-box slot counts when the planner chose perfect-hash indexes (4-byte
-    slots), else None (open addressing: 16-byte slots, capacity pow2 >= 2n)."""
+    slots), else None (open addressing: 16-byte slots, capacity pow2 >= 2n). `clustered`: both
+    build sides verified in key order, indexes positional: the verify pass reads
+    the keys and zeroes the accumulators, nothing is built, no slot is read."""
+    if clustered:
+        return {"q61_shared_scan": 24 * n_ol, "q6_scan_filter_sum": 20 * n_ol, "q1_scan_filter_groupby": 24 * n_ol,
+                "q18_init": 12 * (n_o + n_c) + 16 * n_o,            # verify: keys in, acc zeroed
+                "q18_probe_groupjoin": 20 * n_ol + 16 * n_o + 16 * n_o,
+                "q18_acc_stats": 16 * n_o + 8 * n_o,
+                "q18_having_records": 16 * n_o + 12 * n_o + (4 + 16 + 16) * n_pass,
+                "q18_bucket_scatter": (16 + 16) * n_pass,
+                "q18_bucket_sort_emit": (16 + 40) * n_pass}.get(kernel)
     if box:
         slots_o, slots_c, slot_b = box[0], box[1], 4
     else:
@@ -460,11 +470,12 @@ def main():
             out[name] = (r.device_ms, r.kernels if flags & h.H2TAP_QUERY_PROFILE else [], r.nrows,
                          r.kernel_launches, r.total_rows)
             if name == "q18":
-                dense_seen.append(r.plan_flags == 3)  # both join indexes perfect-hash
+                dense_seen.append(r.plan_flags & 3 == 3)  # both join indexes perfect-hash
+                clustered_seen.append(r.plan_flags >> 3 == 3)  # ... and positional (§4.3)
             h.h2tap_free(r)
         return out
 
-    dense_seen = []
+    dense_seen, clustered_seen = [], []
     dev_flags = h.H2TAP_RESULT_DEVICE
     prof_flags = h.H2TAP_RESULT_DEVICE | h.H2TAP_QUERY_PROFILE
     ALL = tuple(p[0] for p in plans)
@@ -541,6 +552,7 @@ def main():
     value = rows_total / (step_ms / 1e3)
 
     plan_dense = bool(dense_seen) and all(dense_seen)
+    plan_clustered = plan_dense and bool(clustered_seen) and all(clustered_seen)
     # ---- roofline for the dominant kernel (largest share of the step)
     kavg = {k: float(np.mean(v)) for k, v in kern.items()}
     sort_passes = ("v1" if os.environ.get("H2TAP_ORDER") == "v1"
@@ -550,7 +562,8 @@ def main():
     rpeak = read_stream_peak(h, eng, stream) if rank == 0 else None
     roof = None
     if dominant:
-        b = alg_bytes(dominant, n_ol, n_o, n_c, n_pass, sort_passes, box if plan_dense else None)
+        b = alg_bytes(dominant, n_ol, n_o, n_c, n_pass, sort_passes, box if plan_dense else None,
+                      plan_clustered and sort_passes == "carry")
         if b:
             ach = b / (kavg[dominant] / 1e3) / 1e9
             tr = ncu_traffic().get(dominant)
@@ -563,7 +576,8 @@ def main():
                     "timing": "CUDA events on the engine stream, instrumented pass of the same K steps"}
     kernels_summary = {}
     for k, v in kavg.items():
-        b = alg_bytes(k, n_ol, n_o, n_c, n_pass, sort_passes, box if plan_dense else None)
+        b = alg_bytes(k, n_ol, n_o, n_c, n_pass, sort_passes, box if plan_dense else None,
+                      plan_clustered and sort_passes == "carry")
         kernels_summary[k] = {"ms": round(v, 5), "share": round(v / step_ms_local, 4)}
         if b:
             kernels_summary[k]["GB/s"] = round(b / (v / 1e3) / 1e9, 1)
@@ -663,6 +677,8 @@ def main():
             "rows_per_s": dict({f"{q}_in_batch": rows_total / (v / 1e3) for q, v in lat_max.items()},
                                q6_alone=rows_total / (q6_alone_ms / 1e3), q1_alone=rows_total / (q1_alone_ms / 1e3)),
             "q18_result_rows_total": n_pass_total, "q18_result_rows_rank0": n_pass,
+            "q18_join_indexes": ("positional: orders / customer verified in key order on the device (DESIGN.md §4.3)"
+                                 if plan_clustered else "perfect hash" if plan_dense else "hash tables"),
             "roofline": roof,
             "kernels": kernels_summary,
             "cpu_baseline": cpu,

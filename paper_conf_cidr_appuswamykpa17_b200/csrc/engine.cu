@@ -1125,7 +1125,8 @@ JoinIndex plan_index(h2tap_engine *e, const View &v, int table, bool force_hash,
 
 // {nout, err, tie} written by q18_publish (one GPU) or {n_mine, err, tie, -, row0, n_total} by the
 // distributed publish (world > 1), into mapped pinned memory
-struct Q18Small { unsigned long long nout; unsigned int err, tie; Q18Stats st; unsigned long long row0, n_total; };
+struct Q18Small { unsigned long long nout; unsigned int err, tie; Q18Stats st; unsigned long long row0, n_total;
+                  unsigned int clustered; };
 const char *const kQ18Names[8] = {"c_last", "c_id", "o_id", "o_entry_d", "o_ol_cnt", "amount_sum", "o_w_id", "o_d_id"};
 const uint32_t kQ18Types[8] = {H2TAP_I32, H2TAP_I32, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I64, H2TAP_I32, H2TAP_I32};
 const char *const kQ3Names[5] = {"ol_o_id", "ol_w_id", "ol_d_id", "revenue", "o_entry_d"};
@@ -1336,7 +1337,7 @@ void q18_launch_v3(h2tap_engine *e, const View &v, QueryCtx &q) {
                  colp<int32_t>(v, C, H2TAP_C_LAST), q.p[0], s, q.plan_dev, bb, bs, cnt_part, q.out, q.tie_dev,
                  e->num_sms, e->compute, &marks);
     CK(cudaGetLastError());
-    launch_q18_publish(s.nout, s.err, q.tie_dev, q.small_dev, e->compute);  // -> small (mapped)
+    launch_q18_publish(s.nout, s.err, q.tie_dev, q.small_dev, s.jo, s.jc, e->compute);  // -> small (mapped)
 }
 
 // The v3 records did not fit 128 bits (or a bucket overflowed): redo HAVING + ORDER BY on the v2
@@ -1440,7 +1441,7 @@ void q18_gather_and_order(h2tap_engine *e, QueryCtx &q, uint64_t n_rows_max) {
         return;
     }
     q18_sort_and_emit(e, q);
-    launch_q18_publish(s.nout, s.err, q.tie_dev, q.small_dev, e->compute);  // -> small (mapped)
+    launch_q18_publish(s.nout, s.err, q.tie_dev, q.small_dev, s.jo, s.jc, e->compute);  // -> small (mapped)
 }
 
 // ---- NEXT-2: CH Q3 (customer ⋈ new_order ⋈ orders ⋈ order_line) on the Q18 machinery
@@ -1520,6 +1521,7 @@ void finish_q18(h2tap_engine *e, QueryCtx &q) {
         raise(H2TAP_EPLAN, "Q%u: the distributed ORDER BY needs 128-bit carry records; the result "
               "fields are too wide", pl);
     const uint64_t nout = sm->nout;
+    if (!q.dist) r->plan_flags |= (sm->clustered & 3u) << 3;  // bit3 / bit4: positional indexes
     r->total_rows = q.dist ? sm->n_total : nout;
     r->row_offset = q.dist ? sm->row0 : 0;
     if (q.dist && (err & kPeerErrOutCap)) {

@@ -551,21 +551,23 @@ q3_emit_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
     stat.flush(s.stat_part, s.ticket, s.stats);
 }
 
-struct Q18SmallDev { unsigned long long nout; unsigned int err, tie; };  // = engine's Q18Small head
+struct Q18SmallDev { unsigned long long nout; unsigned int err, tie; Q18Stats st; unsigned long long row0, n_total;
+                     unsigned int clustered; };  // = engine's Q18Small
 __global__ void q18_publish_kernel(const unsigned long long *nout, const unsigned int *err,
-                                   const unsigned int *tie, Q18SmallDev *out) {
+                                   const unsigned int *tie, Q18SmallDev *out, JoinIndex jo, JoinIndex jc) {
     pdl_wait();
     pdl_trigger();
     out->nout = *nout;
     out->err = *err;
     out->tie = *tie;
+    out->clustered = (jx_identity(jo) ? 1u : 0u) | (jx_identity(jc) ? 2u : 0u);  // positional indexes used
 }
 
 }  // namespace
 
 void launch_q18_publish(const unsigned long long *nout, const unsigned int *err, const unsigned int *tie,
-                        void *host_small, cudaStream_t st) {
-    launch_pdl(q18_publish_kernel, 1, 1, 0, st, nout, err, tie, static_cast<Q18SmallDev *>(host_small));
+                        void *host_small, const JoinIndex &jo, const JoinIndex &jc, cudaStream_t st) {
+    launch_pdl(q18_publish_kernel, 1, 1, 0, st, nout, err, tie, static_cast<Q18SmallDev *>(host_small), jo, jc);
     count_launches(1);
 }
 

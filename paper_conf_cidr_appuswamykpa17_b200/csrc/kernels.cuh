@@ -198,7 +198,7 @@ void launch_q3_emit(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id,
                     int num_sms, cudaStream_t st);
 // {nout, err, tie} -> mapped pinned host memory (one launch instead of three D2H copies)
 void launch_q18_publish(const unsigned long long *nout, const unsigned int *err, const unsigned int *tie,
-                        void *host_small, cudaStream_t st);
+                        void *host_small, const JoinIndex &jo, const JoinIndex &jc, cudaStream_t st);
 
 // ------------------------------------------------------------------ sort ---
 // Stable LSD radix sort of (u64 key, u32 value) pairs, 8-bit digits, `bits` low key bits.

@@ -347,7 +347,8 @@ def test_q18_planner_dense_and_hash(h, eng, L):
     t = chgen.generate(1, 3, seed=19)
     L.load(t)
     r = h.h2tap_run_query(eng, h.H2TAP_Q18)
-    assert r.plan_flags == 3
+    assert r.plan_flags & 3 == 3
+    assert r.plan_flags >> 3 == 3  # generated tables are in key order: positional indexes (§4.3)
     r.free()
     r = h.h2tap_run_query(eng, h.H2TAP_Q18, flags=HASH)
     assert r.plan_flags == 0
@@ -719,6 +720,10 @@ def test_q18_clustered_index_verification(L, layout, order_mode):
         t["customer"] = {k: v[perm].copy() for k, v in c.items()}
     L.h.h2tap_load_snapshot(L.e, L.h.hot_path_tables(t, (L.h.H2TAP_Q18, L.h.H2TAP_Q3)), L.epoch + 1)
     L.epoch += 1
+    r = L.h.h2tap_run_query(L.e, L.h.H2TAP_Q18)
+    expect = {"clustered": 3, "one_row_swapped": 2, "shuffled": 2, "customer_shuffled": 1}[layout]
+    assert r.plan_flags >> 3 == expect, (layout, r.plan_flags)  # bit3 orders, bit4 customer positional
+    r.free()
     for thr in (Q18_HAVING, 4_000_000):
         want = oracle.q18(t, thr)
         assert_q18(L.q(18, [thr]), want)
