@@ -21,6 +21,8 @@ import numpy as np
 
 _PKG = os.path.dirname(os.path.abspath(__file__))
 LIB_PATH = os.path.join(_PKG, "libh2tap.so")
+if os.environ.get("H2TAP_LIB"):  # an A/B build variant (scripts/build_variants.py), never the default
+    LIB_PATH = os.environ["H2TAP_LIB"]
 
 if not os.path.exists(LIB_PATH):
     raise ImportError(

@@ -208,42 +208,56 @@ __device__ __forceinline__ bool row_less(const Q18Row &x, long long ax, const Q1
 // The key K = a|e|r is unique per result row (r encodes the orders PK), so
 // comparing (hi, lo) as one 128-bit integer is the exact ORDER BY; the payload
 // (c_last, c_id, o_ol_cnt as offsets from their minima) rides in the lowest bits.
-typedef unsigned __int128 u128;
-__device__ __forceinline__ u128 shl128(u128 x, int s) { return s >= 128 ? (u128)0 : x << s; }
-__device__ __forceinline__ u128 shr128(u128 x, int s) { return s >= 128 ? (u128)0 : x >> s; }
-__device__ __forceinline__ unsigned long long lowmask(int b) { return b >= 64 ? ~0ull : (1ull << b) - 1ull; }
-__device__ __forceinline__ unsigned long long shr64(unsigned long long x, int s) { return s >= 64 ? 0ull : x >> s; }
+// Built with 64-bit shifts only: PTX shl / shr clamp shift amounts >= 64 to a zero result, so
+// every field placement is branch-free (an unsigned "negative" amount is >= 64 too). With
+// K = a << (R + E) | e << R | r held as (khi, klo), the record is (K >> L, (K mod 2^L) << P | pay)
+// (L = bits_low, P = payload bits). The u128 formulation it replaced spent ~2x the instructions on
+// variable 128-bit shifts: HAVING 45 -> 40 us, emit 64 -> 56 us measured.
+__device__ __forceinline__ unsigned long long shl_c(unsigned long long x, unsigned s) {
+    unsigned long long r;
+    asm("shl.b64 %0, %1, %2;" : "=l"(r) : "l"(x), "r"(s));
+    return r;
+}
+__device__ __forceinline__ unsigned long long shr_c(unsigned long long x, unsigned s) {
+    unsigned long long r;
+    asm("shr.u64 %0, %1, %2;" : "=l"(r) : "l"(x), "r"(s));
+    return r;
+}
+__device__ __forceinline__ unsigned long long mask_c(unsigned b) { return shr_c(~0ull, 64u - b); }  // b in [0, 64]
 
 __device__ __forceinline__ ulonglong2 carry_record(const Q18Row &r, long long amount, const Q18SortSpec &sp) {
-    const u128 K = shl128((u128)field_a(amount, sp), sp.bits_e + sp.bits_r) |
-                   shl128((u128)field_e(r, sp), sp.bits_r) | (u128)field_r(r, sp);
-    const int P = sp.bits_cl + sp.bits_ci + sp.bits_n;
+    const unsigned R = (unsigned)sp.bits_r, pa = R + (unsigned)sp.bits_e, L = (unsigned)sp.bits_low;
+    const unsigned P = (unsigned)(sp.bits_cl + sp.bits_ci + sp.bits_n);
+    const unsigned long long a = field_a(amount, sp), e = field_e(r, sp), f = field_r(r, sp);
+    const unsigned long long klo = shl_c(a, pa) | shl_c(e, R) | f;  // (R <= 62: e and r start in klo)
+    const unsigned long long khi = shl_c(a, pa - 64u) | shr_c(a, 64u - pa) | shr_c(e, 64u - R);
     const unsigned long long pay =
         (((unsigned long long)((unsigned)r.c_last - (unsigned)sp.cl_min) << sp.bits_ci |
           (unsigned long long)((unsigned)r.c_id - (unsigned)sp.ci_min)) << sp.bits_n) |
         (unsigned long long)((unsigned)r.o_ol_cnt - (unsigned)sp.n_min);
-    const unsigned long long klo = (unsigned long long)K & lowmask(sp.bits_low);
-    return make_ulonglong2((unsigned long long)shr128(K, sp.bits_low),
-                           (unsigned long long)shl128((u128)klo, P) | pay);
+    return make_ulonglong2(shl_c(khi, 64u - L) | shr_c(klo, L), shl_c(klo & mask_c(L), P) | pay);
 }
 
 struct CarryRow { long long amount, o_entry_d; int c_last, c_id, o_id, o_ol_cnt, o_w_id, o_d_id; };
 __device__ __forceinline__ CarryRow carry_decode(unsigned long long hi, unsigned long long lo,
                                                  const Q18SortSpec &sp) {
-    const int P = sp.bits_cl + sp.bits_ci + sp.bits_n;
-    const u128 K = shl128((u128)hi, sp.bits_low) | (u128)(unsigned long long)shr128((u128)lo, P);
-    const unsigned long long fr = (unsigned long long)K & lowmask(sp.bits_r);
-    const unsigned long long fe = (unsigned long long)shr128(K, sp.bits_r) & lowmask(sp.bits_e);
-    const unsigned long long fa = (unsigned long long)shr128(K, sp.bits_r + sp.bits_e);
+    const unsigned R = (unsigned)sp.bits_r, E = (unsigned)sp.bits_e, pa = R + E, L = (unsigned)sp.bits_low;
+    const unsigned bn = (unsigned)sp.bits_n, bci = (unsigned)sp.bits_ci, bo = (unsigned)sp.bits_o,
+                   bd = (unsigned)sp.bits_d;
+    const unsigned P = (unsigned)sp.bits_cl + bci + bn;
+    const unsigned long long klo = shl_c(hi, L) | shr_c(lo, P), khi = shr_c(hi, 64u - L);
+    const unsigned long long fr = klo & mask_c(R);
+    const unsigned long long fe = (shr_c(klo, R) | shl_c(khi, 64u - R)) & mask_c(E);
+    const unsigned long long fa = shr_c(klo, pa) | shl_c(khi, 64u - pa) | shr_c(khi, pa - 64u);
     CarryRow c;
     c.amount = (long long)((unsigned long long)sp.amt_max - fa);
     c.o_entry_d = (long long)((unsigned long long)sp.ent_min + fe);
-    c.o_id = (int)((unsigned)sp.o_min + (unsigned)(fr & lowmask(sp.bits_o)));
-    c.o_d_id = (int)((unsigned)sp.d_min + (unsigned)(shr64(fr, sp.bits_o) & lowmask(sp.bits_d)));
-    c.o_w_id = (int)((unsigned)sp.w_min + (unsigned)shr64(fr, sp.bits_o + sp.bits_d));
-    c.o_ol_cnt = (int)((unsigned)sp.n_min + (unsigned)(lo & lowmask(sp.bits_n)));
-    c.c_id = (int)((unsigned)sp.ci_min + (unsigned)(shr64(lo, sp.bits_n) & lowmask(sp.bits_ci)));
-    c.c_last = (int)((unsigned)sp.cl_min + (unsigned)(shr64(lo, sp.bits_n + sp.bits_ci) & lowmask(sp.bits_cl)));
+    c.o_id = (int)((unsigned)sp.o_min + (unsigned)(fr & mask_c(bo)));
+    c.o_d_id = (int)((unsigned)sp.d_min + (unsigned)(shr_c(fr, bo) & mask_c(bd)));
+    c.o_w_id = (int)((unsigned)sp.w_min + (unsigned)shr_c(fr, bo + bd));
+    c.o_ol_cnt = (int)((unsigned)sp.n_min + (unsigned)(lo & mask_c(bn)));
+    c.c_id = (int)((unsigned)sp.ci_min + (unsigned)(shr_c(lo, bn) & mask_c(bci)));
+    c.c_last = (int)((unsigned)sp.cl_min + (unsigned)(shr_c(lo, bn + bci) & mask_c((unsigned)sp.bits_cl)));
     return c;
 }
 
@@ -1456,19 +1470,22 @@ q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict
     constexpr int U = 4;
     if (s_carry)
     for (uint64_t base = r0; base < r1; base += (uint64_t)U * kHrThreads) {
-        long long sum[U];
-        int w[U], d[U], c[U];
+        long long sum[U], ent[U];
+        int w[U], d[U], c[U], oid[U], cnt[U];
         unsigned int crow[U];
 #pragma unroll
         for (int u = 0; u < U; ++u) {  // independent coalesced loads first
             const uint64_t r = base + (uint64_t)u * kHrThreads + threadIdx.x;
             crow[u] = kNoRow;
             sum[u] = 0; w[u] = d[u] = c[u] = 0;
+            ent[u] = 0; oid[u] = cnt[u] = 0;
             if (r < r1) {
                 const ulonglong2 a = __ldcs(reinterpret_cast<const ulonglong2 *>(s.acc + r));
                 sum[u] = (long long)a.x;
                 crow[u] = ((unsigned int)a.y > 0 && sum[u] > having) ? 0u : kNoRow;
                 w[u] = __ldcs(o_w + r); d[u] = __ldcs(o_d + r); c[u] = __ldcs(o_c + r);
+                // the row's other columns in the same round trip (a row failing HAVING wastes them)
+                ent[u] = __ldcs(o_ent + r); oid[u] = __ldcs(o_id + r); cnt[u] = __ldcs(o_cnt + r);
             }
         }
 #pragma unroll
@@ -1478,13 +1495,12 @@ q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict
 #pragma unroll
         for (int u = 0; u < U; ++u) {
             if (crow[u] == kNoRow) continue;
-            const uint64_t r = base + (uint64_t)u * kHrThreads + threadIdx.x;
             Q18Row row;
-            row.o_entry_d = __ldcs(o_ent + r);
+            row.o_entry_d = ent[u];
             row.c_last = __ldg(c_last + crow[u]);
             row.c_id = c[u];
-            row.o_id = __ldcs(o_id + r);
-            row.o_ol_cnt = __ldcs(o_cnt + r);
+            row.o_id = oid[u];
+            row.o_ol_cnt = cnt[u];
             row.o_w_id = w[u];
             row.o_d_id = d[u];
             rc[u] = carry_record(row, sum[u], sp);
@@ -1515,10 +1531,14 @@ q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict
 __global__ void __launch_bounds__(kObThreads)
 ob_scatter_rec_kernel(const ulonglong2 *__restrict__ rec, uint64_t n_o, const Q18Plan *__restrict__ plan,
                       int nb_launch, const unsigned int *__restrict__ mat, const unsigned int *__restrict__ offset,
-                      const unsigned int *__restrict__ cnt_part, ulonglong2 *__restrict__ kv) {
+                      const unsigned int *__restrict__ cnt_part, ulonglong2 *__restrict__ kv,
+                      unsigned int *big) {
     pdl_wait();
     pdl_trigger();
     extern __shared__ unsigned int cur[];
+    // the emit's oversized-bucket work list (nothing reads it before the emit; a memset node here
+    // would break the PDL chain: -4 us measured); null: the caller resets it
+    if (big && blockIdx.x == 0 && threadIdx.x == 0) *big = 0;
     // (kPeerErrOutCap only stops this rank's emit: its records must still be exchanged)
     if (!plan->spec.carry || (plan->err & ~kPeerErrOutCap)) return;
     const int nb = plan->dist ? (1 << plan->bucket_bits) : nb_launch;
@@ -1592,11 +1612,10 @@ void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, c
     begin("q18_bucket_scatter");
     launch_pdl(ob_scatter_rec_kernel, G, kObThreads, 4 * nb, st, reinterpret_cast<const ulonglong2 *>(bs.k[0]), n_o,
                plan, nb, (const unsigned int *)bs.mat, (const unsigned int *)bs.offset, (const unsigned int *)cnt_part,
-               reinterpret_cast<ulonglong2 *>(bs.kv));
+               reinterpret_cast<ulonglong2 *>(bs.kv), bs.big);
     count_launches(1);
     end();
-    // big[] (the oversized-bucket work list) is reset by the hist kernel on the v2 path
-    cudaMemsetAsync(bs.big, 0, sizeof(unsigned int), st);
+    // (big[], the oversized-bucket work list, was reset by the scatter kernel)
     static const int sub_log2 = [] {
         const char *v = std::getenv("H2TAP_SUB_ROWS_LOG2");
         return v ? std::max(0, std::min(6, std::atoi(v))) : 1;
@@ -1890,7 +1909,7 @@ void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long lo
     if (hv)
         launch_pdl(ob_scatter_rec_kernel, G, kObThreads, nb * 4, st, reinterpret_cast<const ulonglong2 *>(s.k[0]),
                    hv->n_o, (const Q18Plan *)plan, nb, (const unsigned int *)s.mat, (const unsigned int *)s.offset,
-                   (const unsigned int *)hv->cnt_part, reinterpret_cast<ulonglong2 *>(s.kv));
+                   (const unsigned int *)hv->cnt_part, reinterpret_cast<ulonglong2 *>(s.kv), (unsigned int *)nullptr);
     else
         launch_pdl(ob_scatter_kernel, G, kObThreads, nb * 4, st, rows, amt, (const Q18Plan *)plan, nb,
                    (const unsigned int *)s.mat, (const unsigned int *)s.offset, s.kv);

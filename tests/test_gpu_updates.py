@@ -261,6 +261,34 @@ def test_key_column_updates_widen_zone_maps_and_detect_duplicates(h):
         h.h2tap_close(e)
 
 
+def test_entry_and_amount_updates_keep_q18_order_exact(h):
+    """Updates that move o_entry_d far below / above the loaded range and make amounts negative
+    change the ORDER BY plan's field widths (carry records): element-wise parity
+    at several HAVING thresholds, on every epoch."""
+    e = h.h2tap_open(0)
+    try:
+        t = chgen.generate(1, 3, seed=57)
+        t.pop("item")
+        h.h2tap_load_snapshot(e, h.hot_path_tables(t), 1)
+        L = Loader(h, e)
+        o, ol = t["orders"], t["order_line"]
+        rng = np.random.default_rng(57)
+        sel = np.sort(rng.choice(len(o["o_id"]), 6, replace=False)).astype(np.uint32)
+        ent = np.array([o["o_entry_d"].min() - 10 ** 12, o["o_entry_d"].max() + 10 ** 12, -5, 0,
+                        o["o_entry_d"].max() + 1, 1], np.int64)
+        lines = np.sort(rng.choice(len(ol["ol_o_id"]), 500, replace=False)).astype(np.uint32)
+        amt = rng.integers(-10 ** 9, 10 ** 9, size=500).astype(np.int64)
+        for k, upd in enumerate([{"orders": {"o_entry_d": (sel, ent)}},
+                                 {"order_line": {"ol_amount": (lines, amt)}}]):
+            t = oracle.apply_updates(t, upd)
+            h.h2tap_refresh(e, None, upd, 2 + k)
+            L.epoch = 2 + k
+            for having in (Q18_HAVING, -1, -(10 ** 10), int(np.percentile(np.abs(amt), 50))):
+                assert_q18(L.q(18, [having]), oracle.q18(t, having))
+    finally:
+        h.h2tap_close(e)
+
+
 def test_update_errors(h):
     e = h.h2tap_open(0)
     try:
