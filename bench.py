@@ -212,7 +212,8 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None, clustered=F
         return {"q61_shared_scan": 24 * n_ol, "q6_scan_filter_sum": 20 * n_ol, "q1_scan_filter_groupby": 24 * n_ol,
                 "q18_init": 12 * (n_o + n_c) + 16 * n_o,            # verify: keys in, acc zeroed
                 "q18_probe_groupjoin": 20 * n_ol + 16 * n_o + 16 * n_o,
-                "q18_acc_stats": 16 * n_o + 8 * n_o,
+                # one GPU: o_entry_d's bounds come from the snapshot's zone map, acc[] alone is read
+                "q18_acc_stats": 16 * n_o,
                 "q18_having_records": 16 * n_o + 12 * n_o + (4 + 16 + 16) * n_pass,
                 "q18_bucket_scatter": (16 + 16) * n_pass,
                 "q18_bucket_sort_emit": (16 + 40) * n_pass}.get(kernel)
@@ -240,8 +241,8 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None, clustered=F
         "q18_sort_hist": 8 * n_pass,                       # amounts (bucket bits inside field a)
         "q18_bucket_scatter": (16 + 16) * n_pass if sort_passes == "carry"
                               else (40 + 16) * n_pass if sort_passes != "v1" else (12 + 12) * n_pass,
-        # v3 (default): accumulators + o_entry_d of the passing groups for the plan's bounds
-        "q18_acc_stats": 16 * n_o + 8 * n_o,
+        # v3 (default): the accumulators for the plan's amount bounds (o_entry_d: zone map)
+        "q18_acc_stats": 16 * n_o,
         # v3: acc + orders keys in, per result row a customer slot + c_last + (o_id, o_ol_cnt,
         # o_entry_d) and the 16 B carry record out
         "q18_having_records": 16 * n_o + 12 * n_o + (slot_b + 4 + 16 + 16) * n_pass,

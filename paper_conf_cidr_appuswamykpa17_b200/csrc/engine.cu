@@ -237,6 +237,9 @@ inline int stat_col(int table, int slot) {  // column id of a zone-map slot, -1 
     if (table == H2TAP_T_CUSTOMER) return H2TAP_C_LAST;
     return -1;
 }
+// one 64-bit zone-map column per table: orders.o_entry_d, whose range sizes the ORDER BY's entry
+// field (the Q18 plan then reads no o_entry_d column)
+inline int stat64_col(int table) { return table == H2TAP_T_ORDERS ? (int)H2TAP_O_ENTRY_D : -1; }
 inline int stat_slot(int table, uint32_t column) {  // zone-map slot of a column, -1 if none
     for (int s = 0; s < stat_cols(table); ++s)
         if (stat_col(table, s) == (int)column) return s;
@@ -250,6 +253,8 @@ struct View {  // immutable snapshot at one epoch (the paper's shallow-copied to
     // column statistics of the visible rows (zone map): valid once the view is published
     int smin[kTables][kStatCols], smax[kTables][kStatCols];
     bool has_stats[kTables] = {};
+    long long smin64[kTables] = {}, smax64[kTables] = {};  // stat64_col(t)
+    bool has_stats64[kTables] = {};
     // NEXT-4: columns read zero-copy from the caller's pinned host memory (col[][] is then the
     // mapped device address; nothing is kept alive by the view: the caller owns the memory)
     bool host[kTables][kMaxCols] = {};
@@ -286,12 +291,15 @@ struct Pending {
     cudaEvent_t t0, t1, t2, t3;   // timing (copy stream): begin, loads done, update arrays
                                   // uploaded, updates applied
     bool loaded[kTables], full[kTables], updated[kTables];
+    bool stats64_ok[kTables];     // the 64-bit zone map covers every row this refresh loaded
     int *stats_host;              // pinned [kTables][kStatCols][2] delta min/max, then the u64
                                   // count of pages copied into shadows (kStatBytes offset)
     std::pair<void *, size_t> stats_block;
     uint64_t rows_appended, rows_updated, full_copies;
 };
 constexpr size_t kStatBytes = sizeof(int) * kTables * kStatCols * 2;  // multiple of 8
+constexpr size_t kStat64Off = kStatBytes + 8;                          // after the page count
+constexpr size_t kStatTotal = kStat64Off + 16 * kTables;               // + [kTables][2] int64
 
 struct Staging {  // pinned ring for pageable host buffers
     static constexpr size_t kChunk = 32u << 20;
@@ -443,6 +451,20 @@ void publish_ready(h2tap_engine *e, bool wait) {
                     v.smax[t][c] = mx;
                 }
                 v.has_stats[t] = p.loaded[t] || p.updated[t] || carry;
+                if (stat64_col(t) >= 0) {
+                    const long long *d64 = reinterpret_cast<const long long *>(
+                        reinterpret_cast<const char *>(p.stats_host) + kStat64Off) + 2 * t;
+                    const bool carry64 = !p.full[t] && prev && prev->has_stats64[t];
+                    long long mn = INT64_MAX, mx = INT64_MIN;
+                    if (carry64) { mn = prev->smin64[t]; mx = prev->smax64[t]; }
+                    if (p.loaded[t] || p.updated[t]) { mn = std::min(mn, d64[0]); mx = std::max(mx, d64[1]); }
+                    v.smin64[t] = mn;
+                    v.smax64[t] = mx;
+                    // a full reload: the delta covers the table; an append: the previous epoch's
+                    // zone map plus the appended rows; updates widen it (launched per update)
+                    v.has_stats64[t] = v.col[t][stat64_col(t)] && !v.host[t][stat64_col(t)] &&
+                                       (p.full[t] ? p.stats64_ok[t] : carry64 && (!p.loaded[t] || p.stats64_ok[t]));
+                }
             }
         }
         {
@@ -659,13 +681,15 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
     bool must_wait = false;
     Pending pend{};
     pend.epoch = epoch;
-    pend.stats_block = e->host_pool->get(kStatBytes + 8);
+    pend.stats_block = e->host_pool->get(kStatTotal);
     pend.stats_host = static_cast<int *>(pend.stats_block.first);
-    int *stats_dev = static_cast<int *>(e->load_arena.get("load.stats", kStatBytes + 8));
+    int *stats_dev = static_cast<int *>(e->load_arena.get("load.stats", kStatTotal));
+    auto *stats64_dev = reinterpret_cast<long long *>(reinterpret_cast<char *>(stats_dev) + kStat64Off);
     auto *pages_dev = reinterpret_cast<unsigned long long *>(reinterpret_cast<char *>(stats_dev) + kStatBytes);
     for (cudaEvent_t *ev : {&pend.t0, &pend.t1, &pend.t2, &pend.t3}) CK(cudaEventCreate(ev));
     CK(cudaEventRecord(pend.t0, e->copy));
     launch_stats_init(stats_dev, kTables * kStatCols, e->copy);
+    launch_stats_init64(stats64_dev, kTables, e->copy);
     CK(cudaMemsetAsync(pages_dev, 0, 8, e->copy));
     for (uint32_t i = 0; i < ntables; ++i) {
         const h2tap_table &t = tables[i];
@@ -743,6 +767,11 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         pend.loaded[t.table_id] = true;
         pend.full[t.table_id] = full;
         // zone map of the appended rows' key columns, on the copy stream after their H2D
+        if (const int c64 = stat64_col(t.table_id); c64 >= 0 && v->col[t.table_id][c64] && !v->host[t.table_id][c64]) {
+            launch_minmax_i64(static_cast<const int64_t *>(v->col[t.table_id][c64]) + t.first_row,
+                              t.row_count - t.first_row, stats64_dev + 2 * t.table_id, e->num_sms, e->copy);
+            pend.stats64_ok[t.table_id] = true;
+        }
         for (int c = 0; c < stat_cols(t.table_id); ++c)
             if (stat_col(t.table_id, c) >= 0 && v->col[t.table_id][stat_col(t.table_id, c)])
                 launch_minmax_i32(static_cast<const int32_t *>(v->col[t.table_id][stat_col(t.table_id, c)]) + t.first_row,
@@ -800,6 +829,9 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
             const auto *rows_d = reinterpret_cast<const uint32_t *>(upd_dev + upd_off[i]);
             const void *vals_d = upd_dev + upd_off[i] + round_up16(u.n * 4);
             launch_apply_updates(cs.alt->ptr, (uint32_t)es, next_bits, rows_d, vals_d, u.n, e->num_sms, e->copy);
+            if ((int)u.column_id == stat64_col(u.table_id))  // 64-bit zone map: widen
+                launch_minmax_i64(static_cast<const int64_t *>(vals_d), u.n, stats64_dev + 2 * u.table_id,
+                                  e->num_sms, e->copy);
             if (stat_slot(u.table_id, u.column_id) >= 0)  // zone map: widen
                 launch_minmax_i32(static_cast<const int32_t *>(vals_d), u.n,
                                   stats_dev + (u.table_id * kStatCols + stat_slot(u.table_id, u.column_id)) * 2,
@@ -816,7 +848,7 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
     }
     CK(cudaEventRecord(pend.t3, e->copy));
     CK(cudaGetLastError());
-    CK(cudaMemcpyAsync(pend.stats_host, stats_dev, kStatBytes + 8, cudaMemcpyDeviceToHost, e->copy));
+    CK(cudaMemcpyAsync(pend.stats_host, stats_dev, kStatTotal, cudaMemcpyDeviceToHost, e->copy));
     CK(cudaEventCreateWithFlags(&pend.done, cudaEventDisableTiming));
     CK(cudaEventRecord(pend.done, e->copy));
     pend.view = v;
@@ -1262,6 +1294,9 @@ Q18Zone q18_zone(const View &v, bool q3) {
         z.ci_min = v.smin[C][2]; z.ci_max = v.smax[C][2];
         z.n_min = v.smin[O][3]; z.n_max = v.smax[O][3];
     }
+    z.has_e = v.has_stats64[O] ? 1 : 0;
+    z.e_min = v.smin64[O];
+    z.e_max = v.smax64[O];
     return z;
 }
 

@@ -138,6 +138,8 @@ struct Q18Stats {            // min/max of the sort fields that only the result 
 struct Q18Zone {             // bounds of the other result-row fields: the snapshot's zone maps
     int w_min, w_max, d_min, d_max, o_min, o_max;      // orders (w, d, o) key columns
     int cl_min, cl_max, ci_min, ci_max, n_min, n_max;  // c_last, c_id, o_ol_cnt (carry payload)
+    long long e_min, e_max;  // o_entry_d over every orders row (64-bit zone map), valid if has_e
+    int has_e;
 };
 struct __align__(16) Q18Row {  // one result row before ORDER BY: 32 B = one L2 sector per gather
     long long o_entry_d;       // (amount_sum lives in a parallel array: after the sort it is
@@ -350,6 +352,9 @@ void launch_q18_permute(const Q18Row *rows, const long long *amt, const unsigned
 void launch_stats_init(int *out, int n_pairs, cudaStream_t st);
 void launch_gate(unsigned long long ns, cudaStream_t st);  // profiling only  // pairs of (INT_MAX, INT_MIN)
 void launch_minmax_i32(const int32_t *p, uint64_t n, int *out, int num_sms, cudaStream_t st);
+// 64-bit zone map: out[2k] = INT64_MAX, out[2k + 1] = INT64_MIN; then min / max of p[0, n) merged in
+void launch_stats_init64(long long *out, int n_pairs, cudaStream_t st);
+void launch_minmax_i64(const int64_t *p, uint64_t n, long long *out, int num_sms, cudaStream_t st);
 // copy-on-write of updated columns (NEXT-1): page = kCowPageRows rows, one dirty bit per page
 constexpr uint64_t kCowPageRows = 4096;
 static_assert(kCowPageRows * 4 == 4 * 16 * 256, "catch-up kernel: one page = 4/8 uint4 per thread");

@@ -1357,6 +1357,9 @@ q18_acc_stats_kernel(const Q18Acc *__restrict__ acc, const int64_t *__restrict__
     long long amin = INT64_MAX, amax = INT64_MIN, emin = INT64_MAX, emax = INT64_MIN;
     unsigned long long c = 0;
     const uint64_t stride = (uint64_t)gridDim.x * kStatThreads;
+    // with the plan on one GPU the o_entry_d bounds are the snapshot's zone map (every orders row:
+    // a superset of the passing ones): only acc[] is read (48 of 72 MB at W=100)
+    if (make_plan && zone.has_e) o_ent = nullptr;
     constexpr int U = 8;  // independent accumulator loads in flight per thread
     for (uint64_t r0 = (uint64_t)blockIdx.x * kStatThreads + threadIdx.x; r0 < n_o; r0 += U * stride) {
         ulonglong2 a[U];
@@ -1369,7 +1372,7 @@ q18_acc_stats_kernel(const Q18Acc *__restrict__ acc, const int64_t *__restrict__
 #pragma unroll
         for (int u = 0; u < U; ++u) {
             const uint64_t r = r0 + u * stride;
-            e[u] = r < n_o ? __ldcs(o_ent + r) : 0;
+            e[u] = r < n_o && o_ent ? __ldcs(o_ent + r) : 0;
         }
 #pragma unroll
         for (int u = 0; u < U; ++u) {
@@ -1422,6 +1425,7 @@ q18_acc_stats_kernel(const Q18Acc *__restrict__ acc, const int64_t *__restrict__
         g.ent_min = min(g.ent_min, ws[k].ent_min); g.ent_max = max(g.ent_max, ws[k].ent_max);
         gc += wc[k];
     }
+    if (!o_ent) { g.ent_min = zone.e_min; g.ent_max = zone.e_max; }
     *stats = g;
     *count = gc;
     *ticket = 0;  // self-reset

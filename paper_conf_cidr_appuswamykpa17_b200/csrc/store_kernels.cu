@@ -25,6 +25,29 @@ __global__ void stats_init_kernel(int *out, int n_pairs) {
     if (i < n_pairs) { out[2 * i] = INT_MAX; out[2 * i + 1] = INT_MIN; }
 }
 
+__global__ void stats_init64_kernel(long long *out, int n_pairs) {
+    const int i = blockIdx.x * blockDim.x + threadIdx.x;
+    if (i < n_pairs) { out[2 * i] = INT64_MAX; out[2 * i + 1] = INT64_MIN; }
+}
+
+__global__ void __launch_bounds__(256) minmax64_kernel(const int64_t *__restrict__ p, uint64_t n, long long *out) {
+    long long mn = INT64_MAX, mx = INT64_MIN;
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
+        const long long v = __ldcs(reinterpret_cast<const long long *>(p) + i);
+        mn = min(mn, v);
+        mx = max(mx, v);
+    }
+    for (int o = 16; o; o >>= 1) {
+        mn = min(mn, __shfl_xor_sync(0xffffffffu, mn, o));
+        mx = max(mx, __shfl_xor_sync(0xffffffffu, mx, o));
+    }
+    if ((threadIdx.x & 31) == 0 && mn <= mx) {
+        atomicMin(out, mn);
+        atomicMax(out + 1, mx);
+    }
+}
+
 __global__ void __launch_bounds__(256) minmax_kernel(const int32_t *__restrict__ p, uint64_t n, int *out) {
     int mn = INT_MAX, mx = INT_MIN;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
@@ -159,6 +182,18 @@ void launch_stats_init(int *out, int n_pairs, cudaStream_t st) {
     stats_init_kernel<<<(n_pairs + 127) / 128, 128, 0, st>>>(out, n_pairs);
 }
 
+void launch_stats_init64(long long *out, int n_pairs, cudaStream_t st) {
+    stats_init64_kernel<<<(n_pairs + 127) / 128, 128, 0, st>>>(out, n_pairs);
+}
+
+void launch_minmax_i64(const int64_t *p, uint64_t n, long long *out, int num_sms, cudaStream_t st) {
+    if (!n) return;
+    uint64_t blocks = (n + 255) / 256;
+    const uint64_t cap = (uint64_t)num_sms * 4;
+    if (blocks > cap) blocks = cap;
+    minmax64_kernel<<<(unsigned)blocks, 256, 0, st>>>(p, n, out);
+}
+
 void launch_minmax_i32(const int32_t *p, uint64_t n, int *out, int num_sms, cudaStream_t st) {
     if (!n) return;
     uint64_t blocks = (n + 255) / 256;
@@ -188,7 +223,7 @@ cudaError_t set_attributes_store(int num_sms) {
         (const void *)cow_catchup_kernel<8>,
         (const void *)gate_kernel,
         (const void *)minmax_kernel,
-        (const void *)stats_init_kernel};
+        (const void *)stats_init_kernel, (const void *)stats_init64_kernel, (const void *)minmax64_kernel};
     const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
     if (le != cudaSuccess) return le;
     return cudaSuccess;
