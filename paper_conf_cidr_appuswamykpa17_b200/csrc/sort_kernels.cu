@@ -24,6 +24,18 @@
 #include "kernels.cuh"
 #include "peer.cuh"
 
+// per-bucket emit geometry (A/B via scripts/build_variants.py): carry-record capacity of the small
+// instance, its blocks per SM, and the row-id path's capacity (both share its shared memory)
+#ifndef OB_CAP
+#define OB_CAP 1536
+#endif
+#ifndef EMIT_BPS
+#define EMIT_BPS 6
+#endif
+#ifndef ROW_CAP
+#define ROW_CAP 1024
+#endif
+
 namespace h2tap {
 namespace {
 
@@ -455,7 +467,10 @@ constexpr int kBkThreads = 256;
 constexpr int kBkItems = 16;                       // rows per thread in the scatter
 constexpr int kLsCapSmall = 2048;                  // rows per bucket: v1 small instance
 constexpr int kLsCapLarge = 8192;                  // rows per bucket: large-bucket kernel
-constexpr int kLsSubMax = 512;                     // max sub-buckets per bucket (4 per emit thread)
+#ifndef LS_SUB_MAX
+#define LS_SUB_MAX 512
+#endif
+constexpr int kLsSubMax = LS_SUB_MAX;              // max sub-buckets per bucket (4 per emit thread)
 constexpr int kEmThreads = 128;                    // per-bucket sort / emit block (8 blocks/SM)
 
 // 1. keys + histogram (+ bucket scan by the last block)
@@ -764,7 +779,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
 // capacity in big[1..]; the large instance walks only that queue.
 // kPairs: k holds interleaved 16-byte (key, row id) pairs (v2 scatter), v is unused.
 template <int kLsCap, int kMin, bool kPairs = false>
-__global__ void __launch_bounds__(kEmThreads, 6)
+__global__ void __launch_bounds__(kEmThreads, EMIT_BPS)
 bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigned int *__restrict__ v,
                          const unsigned int *__restrict__ offset, int nb,
                          const Q18Plan *__restrict__ plan, const Q18Row *__restrict__ rows,
@@ -788,7 +803,7 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
     // row-id path: the v2 small instance holds 1 024 rows (LsSmem<1024> fits the 35 KB of the
     // carry layout, so both run 6 blocks per SM); larger buckets go to the large instance
     if (rows == nullptr) return;  // v3 / distributed: carry records only (row path re-run by the host)
-    constexpr int kRowCap = (kPairs && kMin == 0) ? 1024 : kLsCap;
+    constexpr int kRowCap = (kPairs && kMin == 0) ? ROW_CAP : kLsCap;
     LsSmem<kRowCap> &S = *reinterpret_cast<LsSmem<kRowCap> *>(smem_raw);
     const int shift = plan->shift;
     const Q18SortSpec sp = plan->spec;
@@ -994,11 +1009,11 @@ carry_large_emit_kernel(const unsigned long long *__restrict__ k, const unsigned
 // scattered 40 B/row writes cost more than the random gather they save) and sorting chunks of
 // whole buckets per block (fewer barriers, but 2 blocks/SM left the gathers latency-bound).
 constexpr int kObThreads = 1024;   // hist / scatter: 2 blocks of 32 warps per SM
-constexpr int kObCap = 1536;  // per-bucket sort capacity (carry: 35 KB, 6 blocks of 128 threads/SM);
+constexpr int kObCap = OB_CAP;  // per-bucket sort capacity (carry: 35 KB, 6 blocks of 128 threads/SM);
                                      // 4 096 (2 blocks/SM) with ~730-row buckets measured slower
 // dynamic shared memory of the v2 emit instances: row-id or carry layout, whichever is larger
-constexpr size_t kObSmem = sizeof(LsSmem<1024>) > sizeof(LcSmem<kObCap>) ? sizeof(LsSmem<1024>)
-                                                                         : sizeof(LcSmem<kObCap>);
+constexpr size_t kObSmem = sizeof(LsSmem<ROW_CAP>) > sizeof(LcSmem<kObCap>) ? sizeof(LsSmem<ROW_CAP>)
+                                                                            : sizeof(LcSmem<kObCap>);
 constexpr size_t kObSmemLarge = sizeof(LsSmem<kLsCapLarge>) > sizeof(LcSmem<kLcCapLarge>)
                                     ? sizeof(LsSmem<kLsCapLarge>) : sizeof(LcSmem<kLcCapLarge>);
 
@@ -1625,7 +1640,7 @@ void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, c
         return v ? std::max(0, std::min(6, std::atoi(v))) : 1;
     }();
     begin("q18_bucket_sort_emit");
-    const unsigned lb = (unsigned)nb < (unsigned)num_sms * 6 ? (unsigned)nb : (unsigned)num_sms * 6;
+    const unsigned lb = (unsigned)nb < (unsigned)num_sms * EMIT_BPS ? (unsigned)nb : (unsigned)num_sms * EMIT_BPS;
     launch_pdl(bucket_local_emit_kernel<kObCap, 0, true>, lb, kEmThreads, kObSmem, st,
                (const unsigned long long *)bs.kv, (const unsigned int *)nullptr, (const unsigned int *)bs.offset, nb,
                plan, (const Q18Row *)nullptr, (const long long *)nullptr, dst, flag, bs.big, sub_log2, PeerArgs{});
