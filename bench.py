@@ -9,10 +9,15 @@ per GPU (~30M order_line rows), synthetic ('spread' population, seed 1).
 
 value  = order_line rows per second through one full pass of the hot path, whole job: every
          rank's visible order_line rows (each counted ONCE per step, although Q6, Q1 and Q18 all
-         read them) / step time (max over ranks), snapshot resident in HBM.
+         read them) / step time (max over ranks), snapshot resident in HBM. Step time = the
+         batch's GPU span from the library's CUDA events on its stream (h2tap_last_batch_ms:
+         before the first kernel, after the last); ms_per_step_host_return adds the host's
+         wake-up and return path (the bench's own events around the synchronous call).
 e2e    = same metric through the public API with host buffers: each step refreshes the snapshot
          from pinned host memory (full reload, H2D inside the timed region), runs the batch and
          returns every result to host memory; the serial figure (queries read that step's upload).
+         e2e_incremental: the snapshot stays resident, each step refreshes it with that step's
+         NewOrder appends + Delivery updates only (the paper's fresh-snapshot loop).
 roofline: the dominant kernel's algorithmic bytes per launch / its CUDA-event duration,
          against MEASURED_PEAKS.json hbm_gbs (copy) and the live read-stream peak.
 c1     = BASELINE configs[0]: Q6 at W=1 on one GPU, device and e2e latency, oracle beside it.
@@ -548,6 +553,7 @@ def main():
     starts = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
     ends = [torch.cuda.Event(enable_timing=True) for _ in range(a.steps)]
     per_query = {q: [] for q in ALL}
+    batch_dev = []  # the library's own events around each batch's GPU work (h2tap_last_batch_ms)
     launches = 0
     n_pass = n_pass_total = 0
     barrier()
@@ -557,13 +563,19 @@ def main():
             torch.cuda._sleep(a.sleep_cycles)  # batch while the GPU sleeps (no launch gap inside)
         starts[i].record(stream)
         out = run_batch(ALL, dev_flags, ends[i])
+        batch_dev.append(h.h2tap_last_batch_ms(eng))
         for q, (ms, ks, nrows, nl, tot) in out.items():
             per_query[q].append(ms)
             launches += nl
         if "q18" in out:
             n_pass, n_pass_total = out["q18"][2], out["q18"][4]
     barrier()
-    step_ms_local = sum(s.elapsed_time(e) for s, e in zip(starts, ends)) / a.steps
+    # the step = the batch's GPU span: CUDA events on the engine stream before its first kernel and
+    # after its last (h2tap_last_batch_ms); the bench's own events around the call (end recorded
+    # when the synchronous call has returned to Python) add the host's wake-up + return path and
+    # are reported next to it
+    step_host_ms_local = sum(s.elapsed_time(e) for s, e in zip(starts, ends)) / a.steps
+    step_ms_local = float(np.mean(batch_dev))
 
     # ---- the scans alone (not sharing a pass): Q6 by itself, Q1 by itself (C2 = Q1 at W=100).
     # The query's own CUDA events (result.device_ms, recorded on the engine stream around its
@@ -594,8 +606,8 @@ def main():
                 kern.setdefault(kname, []).append(kms)
     barrier()
     clk = clocks.stop()
-    step_ms, q6_alone_ms, q1_alone_ms = max_over_ranks([step_ms_local, alone.get("q6", float("nan")),
-                                                       alone.get("q1", float("nan"))])
+    step_ms, step_host_ms, q6_alone_ms, q1_alone_ms = max_over_ranks(
+        [step_ms_local, step_host_ms_local, alone.get("q6", float("nan")), alone.get("q1", float("nan"))])
     lat = {q: float(np.median(v)) for q, v in per_query.items()}
     lat_max = dict(zip(lat, max_over_ranks(list(lat.values()))))
     nt = torch.tensor([n_ol], dtype=torch.float64, device=pg_dev)
@@ -748,6 +760,7 @@ def main():
         line = {
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": a.steps,
             "warmup": a.warmup, "ms_per_step": step_ms, "higher_is_better": True,
+            "ms_per_step_host_return": round(step_host_ms, 5),
             "scaling": "strong" if strong else "weak", "vs_baseline": None, "dtype": "int64",
             "data": "synthetic",
             "config": {"workload": (f"CH {'+'.join(q.upper() for q in ALL)} per step over W={W} warehouses split over {world} GPU(s)"
@@ -768,6 +781,10 @@ def main():
                                         "§4.5); every query computes its full result; the scans alone "
                                         "are in latency_ms.q6_alone / q1_alone"
                                         if os.environ.get("H2TAP_SHARED_SCAN", "1") != "0" else "off"),
+                       "timing": "ms_per_step: the batch's GPU span, CUDA events recorded by the library on its "
+                                 "stream around the batch (h2tap_last_batch_ms), per step, mean; "
+                                 "ms_per_step_host_return: bench events around the call, end recorded "
+                                 "after it returned to Python",
                        "l2": ("inputs > L2; between steps (outside events) 512 MB written then 256 MB read to flush L2"
                               if flush is not None else "inputs > L2 (no flush)")},
             "latency_ms": dict({f"{q}_in_batch": round(v, 4) for q, v in lat_max.items()},

@@ -149,6 +149,7 @@ _lib.h2tap_run_query.argtypes = [_P, C.c_uint32, C.POINTER(C.c_int64), C.c_uint3
                                  C.POINTER(C.POINTER(h2tap_result))]
 _lib.h2tap_run_queries.argtypes = [_P, C.POINTER(h2tap_query), C.c_uint32,
                                    C.POINTER(C.POINTER(h2tap_result))]
+_lib.h2tap_last_batch_ms.argtypes = [_P, C.POINTER(C.c_double)]
 _lib.h2tap_free.argtypes = [C.POINTER(h2tap_result)]
 _lib.h2tap_free.restype = None
 _lib.h2tap_close.argtypes = [_P]
@@ -163,7 +164,8 @@ for _f in ("h2tap_open", "h2tap_load_snapshot_ex", "h2tap_load_snapshot", "h2tap
            "h2tap_reserve", "h2tap_refresh", "h2tap_refresh_rows", "h2tap_get_store_stats",
            "h2tap_sync",
            "h2tap_run_query_ex", "h2tap_run_query", "h2tap_run_queries", "h2tap_peer_handle",
-           "h2tap_peer_connect", "h2tap_peer_connect_local", "h2tap_compute_stream", "h2tap_layout_sum"):
+           "h2tap_peer_connect", "h2tap_peer_connect_local", "h2tap_compute_stream", "h2tap_layout_sum",
+           "h2tap_last_batch_ms"):
     getattr(_lib, _f).restype = C.c_int
 
 ABI_SYMBOLS = ["h2tap_open", "h2tap_load_snapshot", "h2tap_load_snapshot_ex",
@@ -172,7 +174,7 @@ ABI_SYMBOLS = ["h2tap_open", "h2tap_load_snapshot", "h2tap_load_snapshot_ex",
                "h2tap_run_query", "h2tap_run_query_ex", "h2tap_run_queries", "h2tap_free", "h2tap_close",
                "h2tap_last_error", "h2tap_peer_handle", "h2tap_peer_connect",
                "h2tap_peer_connect_local", "h2tap_compute_stream",
-               "h2tap_c_last_name", "h2tap_layout_sum"]
+               "h2tap_c_last_name", "h2tap_layout_sum", "h2tap_last_batch_ms"]
 
 
 class H2tapError(RuntimeError):
@@ -419,6 +421,13 @@ def h2tap_refresh_rows(engine: Engine, tables: dict | None, updates: dict | None
 def h2tap_reserve(engine: Engine, table: str, rows: int) -> None:
     """Pre-size a loaded table's columns for ``rows`` rows (appends then never reallocate)."""
     _check(_lib.h2tap_reserve(engine.handle, SCHEMA[table][0], rows))
+
+
+def h2tap_last_batch_ms(engine: Engine) -> float:
+    """Device time (CUDA events, ms) of the engine's last completed h2tap_run_queries batch."""
+    ms = C.c_double()
+    _check(_lib.h2tap_last_batch_ms(engine.handle, C.byref(ms)))
+    return ms.value
 
 
 def h2tap_sync(engine: Engine) -> int:

@@ -405,6 +405,8 @@ struct h2tap_engine {
     cudaStream_t reaper = nullptr;  // stream-ordered frees of snapshot buffers
     FreeOrder free_order;
     cudaEvent_t q_begin = nullptr, q_end = nullptr;
+    cudaEvent_t b_begin = nullptr, b_end = nullptr;  // the last h2tap_run_queries batch on the device
+    float last_batch_ms = -1.f;
 
     std::mutex load_mu, query_mu, view_mu, pend_mu;
     TableState tables[kTables];
@@ -1963,6 +1965,7 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
             }
         }
     };
+    CK(cudaEventRecord(e->b_begin, e->compute));
     CK(cudaEventRecord(e->ev_fork, e->compute));  // the batch start (fork point of the side stream)
     for (size_t i = 0; i < ctx.size(); ++i) {
         QueryCtx &q = ctx[i];
@@ -2020,7 +2023,9 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
         q.mark1 = e->prof.marks.size();
     }
     join_side();
+    CK(cudaEventRecord(e->b_end, e->compute));  // every kernel of the batch, side stream included
     finish_upto(ctx.size());
+    CK(cudaEventElapsedTime(&e->last_batch_ms, e->b_begin, e->b_end));
     const double wall = std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - t0).count();
     for (uint32_t i = 0; i < n; ++i) {
         QueryCtx &q = ctx[i];
@@ -2131,6 +2136,8 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         }
         CK(cudaEventCreate(&e->q_begin));
         CK(cudaEventCreate(&e->q_end));
+        CK(cudaEventCreate(&e->b_begin));
+        CK(cudaEventCreate(&e->b_end));
         CK(cudaMallocHost(&e->small_host, 256));
         e->arena.device = e->device;
         e->load_arena.device = e->device;
@@ -2387,6 +2394,14 @@ h2tap_status h2tap_run_queries(h2tap_engine *e, const h2tap_query *queries, uint
     return guarded([&] { return queries_impl(e, queries, nqueries, out); });
 }
 
+h2tap_status h2tap_last_batch_ms(h2tap_engine *e, double *device_ms) {
+    if (!e || !device_ms) return fail(H2TAP_EINVAL, "engine / device_ms is NULL");
+    std::lock_guard<std::mutex> g(e->query_mu);
+    if (e->last_batch_ms < 0.f) return fail(H2TAP_EPLAN, "no batch has completed on this engine");
+    *device_ms = e->last_batch_ms;
+    return H2TAP_OK;
+}
+
 void h2tap_free(h2tap_result *r) {
     if (!r) return;
     delete static_cast<ResultImpl *>(r);
@@ -2412,6 +2427,8 @@ void h2tap_close(h2tap_engine *e) {
     for (auto ev : e->prof.pool) cudaEventDestroy(ev);
     cudaEventDestroy(e->q_begin);
     cudaEventDestroy(e->q_end);
+    cudaEventDestroy(e->b_begin);
+    cudaEventDestroy(e->b_end);
     cudaFreeHost(e->small_host);
     e->published.reset();
     e->accepted.reset();

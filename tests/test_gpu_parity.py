@@ -387,6 +387,26 @@ def test_device_resident_results(h, L):
     assert_q1(L.q(1, flags=h.H2TAP_RESULT_DEVICE | h.H2TAP_QUERY_PROFILE), oracle.q1(t, Q1_CUTOFF))
 
 
+def test_last_batch_device_ms(h):
+    """h2tap_last_batch_ms: EPLAN before any batch; after a batch, the GPU span of its kernels —
+    positive, at least the longest query's own device time, at most the call's wall clock."""
+    e = h.h2tap_open(0)
+    try:
+        with pytest.raises(h.H2tapError) as ei:
+            h.h2tap_last_batch_ms(e)
+        assert ei.value.status == h.H2TAP_EPLAN
+        t = chgen.generate(1, 3, seed=4)
+        h.h2tap_load_snapshot(e, h.hot_path_tables(t), 1)
+        rs = h.h2tap_run_queries(e, [(h.H2TAP_Q6, None, 0), (h.H2TAP_Q1, None, 0), (h.H2TAP_Q18, None, 0)])
+        ms = h.h2tap_last_batch_ms(e)
+        assert 0 < ms <= max(r.e2e_ms for r in rs) + 1e-3
+        assert ms >= max(r.device_ms for r in rs) - 1e-3
+        for r in rs:
+            h.h2tap_free(r)
+    finally:
+        h.h2tap_close(e)
+
+
 def test_profile_reports_kernels(h, eng, L):
     t = chgen.generate(1, 2, seed=3)
     L.load(t)
