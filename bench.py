@@ -581,8 +581,8 @@ def main():
     # The query's own CUDA events (result.device_ms, recorded on the engine stream around its
     # kernels); a ~50 us sleep kernel queued first lets the host enqueue the whole query before the
     # GPU reaches it, so no launch latency lands inside the window
-    alone = {}
-    for q in [x for x in ("q6", "q1") if x in ALL]:
+    alone, alone_p99 = {}, {}
+    for q in [x for x in ("q6", "q1", "q18") if x in ALL]:  # (Q18 alone: config C3)
         for _ in range(2):
             run_batch((q,), dev_flags)
         barrier()
@@ -593,6 +593,25 @@ def main():
                 torch.cuda._sleep(a.sleep_cycles)
             ms.append(run_batch((q,), dev_flags)[q][0])
         alone[q] = float(np.median(ms))
+        alone_p99[q] = float(np.percentile(ms, 99))
+    barrier()
+    # C3 end to end: Q18 alone with its result rows copied to host memory (the D2H of the result
+    # columns is inside; its bytes are reported), host wall clock around the call, median
+    c3_e2e_ms = c3_d2h = None
+    if "q18" in ALL:
+        c3 = []
+        for k in range(3 + min(a.steps, 10)):
+            flush_l2()
+            torch.cuda.synchronize()
+            t0 = time.perf_counter()
+            r = h.h2tap_run_query(eng, h.H2TAP_Q18, Q18_P)  # host result: columns in host memory
+            _ = r.columns["amount_sum"][:1].sum() if r.nrows else 0  # host read
+            dt = (time.perf_counter() - t0) * 1e3
+            c3_d2h = int(sum(v.nbytes for v in r.columns.values()))
+            h.h2tap_free(r)
+            if k >= 3:
+                c3.append(dt)
+        c3_e2e_ms = float(np.median(c3))
     barrier()
 
     # ---- instrumented pass (same K steps): per-kernel CUDA events for the roofline; a 30 us gate
@@ -606,8 +625,9 @@ def main():
                 kern.setdefault(kname, []).append(kms)
     barrier()
     clk = clocks.stop()
-    step_ms, step_host_ms, q6_alone_ms, q1_alone_ms = max_over_ranks(
-        [step_ms_local, step_host_ms_local, alone.get("q6", float("nan")), alone.get("q1", float("nan"))])
+    step_ms, step_host_ms, q6_alone_ms, q1_alone_ms, q18_alone_ms, step_p50, step_p99 = max_over_ranks(
+        [step_ms_local, step_host_ms_local, alone.get("q6", float("nan")), alone.get("q1", float("nan")),
+         alone.get("q18", float("nan")), float(np.median(batch_dev)), float(np.percentile(batch_dev, 99))])
     lat = {q: float(np.median(v)) for q, v in per_query.items()}
     lat_max = dict(zip(lat, max_over_ranks(list(lat.values()))))
     nt = torch.tensor([n_ol], dtype=torch.float64, device=pg_dev)
@@ -640,10 +660,13 @@ def main():
                     "frac_of_read_stream_peak": round(ach / rpeak, 4) if rpeak else None,
                     "timing": "CUDA events on the engine stream, instrumented pass of the same K steps"}
     kernels_summary = {}
+    q18_alg = 0
     for k, v in kavg.items():
         b = alg_bytes(k, n_ol, n_o, n_c, n_pass, sort_passes, box if plan_dense else None,
                       plan_clustered and sort_passes == "carry")
         kernels_summary[k] = {"ms": round(v, 5), "share": round(v / step_ms_local, 4)}
+        if b and k.startswith("q18"):
+            q18_alg += int(b)
         if b:
             kernels_summary[k]["GB/s"] = round(b / (v / 1e3) / 1e9, 1)
             kernels_summary[k]["frac_hbm"] = round(b / (v / 1e3) / 1e9 / peak, 4)
@@ -791,6 +814,27 @@ def main():
                                q6_alone=round(q6_alone_ms, 4), q1_alone=round(q1_alone_ms, 4),
                                **({"q6_q1_shared_scan_batch": round(lat_max["q6"] + lat_max["q1"], 4)}
                                   if "q6" in lat_max and "q1" in lat_max else {})),
+            "step_ms_median": round(step_p50, 5), "step_ms_p99": round(step_p99, 5),
+            "c2": ({"workload": "CH Q1 alone at W=100 per GPU (BASELINE configs[1]), device time (query's own events), "
+                               "median / p99 of the K steps", "latency_ms": round(q1_alone_ms, 4),
+                    "latency_p99_ms": round(alone_p99.get("q1", float("nan")), 4),
+                    "rows_per_s": rows_total / (q1_alone_ms / 1e3),
+                    "GB/s": round(24 * n_ol / (q1_alone_ms / 1e3) / 1e9, 1),
+                    "frac_of_8TBps": round(24 * n_ol / (q1_alone_ms / 1e3) / 8.0e12, 4),
+                    "frac_of_measured_peak": round(24 * n_ol / (q1_alone_ms / 1e3) / 1e9 / peak, 4),
+                    "target": "kernel <= 129 us (>= 70 % of 8 TB/s), SURVEY.md §8(d)"} if "q1" in ALL else None),
+            "c3": ({"workload": "CH Q18 alone at W=100 per GPU (BASELINE configs[2]), 1 GPU",
+                    "device_ms": round(q18_alone_ms, 4), "device_p99_ms": round(alone_p99.get("q18", float("nan")), 4),
+                    "e2e_ms": round(c3_e2e_ms, 3) if c3_e2e_ms else None, "e2e_d2h_bytes": c3_d2h,
+                    "e2e_how": "h2tap_run_query with a host result (the result columns' D2H inside), host wall "
+                               "clock around the call, median",
+                    "result_rows": n_pass_total,
+                    "algorithmic_bytes": q18_alg,
+                    "GB/s_on_algorithmic_bytes": round(q18_alg / (q18_alone_ms / 1e3) / 1e9, 1) if q18_alg else None,
+                    "frac_of_measured_peak": round(q18_alg / (q18_alone_ms / 1e3) / 1e9 / peak, 4) if q18_alg else None,
+                    "frac_of_8TBps": round(q18_alg / (q18_alone_ms / 1e3) / 8.0e12, 4) if q18_alg else None,
+                    "bytes_model": "sum of the Q18 kernels' algorithmic bytes (bench.py alg_bytes, DESIGN.md §5)"}
+                   if "q18" in ALL and world == 1 else None),
             "rows_per_s": dict({f"{q}_in_batch": rows_total / (v / 1e3) for q, v in lat_max.items()},
                                q6_alone=rows_total / (q6_alone_ms / 1e3), q1_alone=rows_total / (q1_alone_ms / 1e3)),
             "q18_result_rows_total": n_pass_total, "q18_result_rows_rank0": n_pass,

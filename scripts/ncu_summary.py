@@ -34,7 +34,10 @@ if os.path.exists(rp):
     want = ["Kernel Name", "gpu__time_duration.sum", "dram__bytes_read.sum", "dram__bytes_write.sum",
             "gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed",
             "sm__throughput.avg.pct_of_peak_sustained_elapsed", "launch__registers_per_thread",
-            "sm__warps_active.avg.pct_of_peak_sustained_active", "lts__t_sector_hit_rate.pct"]
+            "sm__warps_active.avg.pct_of_peak_sustained_active", "lts__t_sector_hit_rate.pct",
+            # SURVEY.md §8(d) timing protocol's list: shared atomics, global load sectors, issue
+            "smsp__inst_executed_op_shared_atom.sum", "l1tex__t_sectors_pipe_lsu_mem_global_op_ld.sum",
+            "smsp__issue_active.avg.pct_of_peak_sustained_active", "smsp__inst_executed.sum"]
     idx = [h.index(w) for w in want if w in h]
     out.append(f"\n## ncu --set full ({rp.split('/')[-1]})\n")
     out.append("| " + " | ".join(h[i] for i in idx) + " |")
