@@ -165,6 +165,19 @@ def test_boundaries_fixture(L, order_mode):
             assert list(zip(*[got[k].tolist() for k in Q18_NAMES])) == want, case["_why"]
 
 
+def test_q18_tiebreak_fixture(L, order_mode):
+    """tests/golden/tiebreak_q18.json: four groups tied on (amount_sum, o_entry_d) in different
+    warehouses and districts, ordered by o_w_id, o_d_id, o_id (R33); hand-derived."""
+    t, exp = golden("tiebreak_q18.json")
+    L.load(t)
+    for case in exp["q18"]:
+        for flags in (0, HASH):
+            got = L.q(18, case["params"], flags=flags)
+            want = [(r["c_last"], r["c_id"], r["o_id"], iso_us(r["o_entry_d"]), r["o_ol_cnt"],
+                     r["amount_sum"], r["o_w_id"], r["o_d_id"]) for r in case["rows"]]
+            assert list(zip(*[got[k].tolist() for k in Q18_NAMES])) == want, case["_why"]
+
+
 def test_q18_having_exactly_at_group_sums(L, order_mode):
     """HAVING thresholds equal to existing group sums (the '>' boundary) at W=2: the group at the
     threshold is excluded, the one 1 cent above it included, on both join-index layouts."""

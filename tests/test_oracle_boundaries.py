@@ -8,7 +8,8 @@ SQLite running the literal CH SQL on the same rows:
   * Q1  ``ol_delivery_d > cutoff`` (strict);
   * Q18 ``HAVING SUM(ol_amount) > 200`` (strict; a group summing to exactly the threshold is out);
   * NULL dates (R5) against constants equal to the sentinel's own value INT64_MIN.
-The mutations these catch (each fails at least one test here): HAVING '>' -> '>=',
+Also the Q18 tie-break (tests/golden/tiebreak_q18.json: ties on (amount_sum, o_entry_d) across
+warehouses and districts). The mutations these catch (each fails at least one test here): HAVING '>' -> '>=',
 Q6 '<' -> '<=' on d_hi, '>=' -> '>' on d_lo, Q1 '>' -> '>=', BETWEEN made exclusive, and a NULL
 test dropped from any one of the 3-valued comparison helpers (pinned against SQLite directly,
 because inside Q6 a dropped NULL test in one helper is masked by the other's UNKNOWN).
@@ -102,6 +103,22 @@ def test_boundaries_fixture_vs_sqlite_and_brute_force():
     for case in exp["q18"]:
         assert sqlite_q18(db, case["params"][0]) == want_q18(case), case["_why"]
         assert brute_q18(t, case["params"][0]) == want_q18(case), case["_why"]
+
+
+def test_q18_tiebreak_golden():
+    """tests/golden/tiebreak_q18.json (hand-derived): rows tied on (amount_sum, o_entry_d) come in
+    (o_w_id, o_d_id, o_id) order (R33). The brute-force evaluation implements the same
+    reading; SQLite runs the literal CH SQL, whose ORDER BY stops at o_entry_d, so it fixes the
+    sequence of (amount_sum, o_entry_d) and the row set, not the order inside a tie."""
+    t, exp = golden("tiebreak_q18.json")
+    db = sqlite_load(t)
+    for case in exp["q18"]:
+        want = want_q18(case)
+        assert q18_tuples(oracle.q18(t, case["params"][0])) == want, case["_why"]
+        assert brute_q18(t, case["params"][0]) == want, case["_why"]
+        lite = sqlite_q18(db, case["params"][0])
+        assert sorted(lite) == sorted(want)
+        assert [(r[5], r[3]) for r in lite] == [(r[5], r[3]) for r in want]
 
 
 @pytest.mark.parametrize("op", [">=", "<", ">"])

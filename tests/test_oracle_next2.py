@@ -70,6 +70,33 @@ def test_golden_fixture():
     assert [list(x) for x in zip(r4["o_ol_cnt"].tolist(), r4["order_count"].tolist())] == want["q4"]
 
 
+def test_golden_fixture_vs_sqlite_and_brute_force():
+    """The hand-derived Q4 / Q12 groups of the fixture (incl. orders entered exactly at Q4's
+    window bounds) are also what SQLite's CH SQL and the nested loops give."""
+    t, p, want = golden_next2()
+    db = sqlite_load(t)
+    assert [list(r) for r in sqlite_q4(db, *p["q4"])] == want["q4"]
+    assert [list(r) for r in brute_q4(t, *p["q4"])] == want["q4"]
+    assert [list(r) for r in sqlite_q12(db, *p["q12"])] == want["q12"]
+    assert [list(r) for r in brute_q12(t, *p["q12"])] == want["q12"]
+
+
+def test_q14_prefix_longer_than_the_column():
+    """LIKE 'p%' with p longer than the fixed-width i_data value matches nothing (the value is too
+    short to start with p): a 50-byte i_data followed in memory by a row starting with the
+    pattern's 51st character must not match."""
+    t, p, _ = golden_next2()
+    d50 = b"PR" + b"x" * 48
+    t["item"] = {"i_id": np.array([1, 2, 3], np.int32),
+                 "i_data": np.array([d50, b"Yzz", b"XPR"], dtype="S50")}
+    r = oracle.q14(t, *p["q14"][:2], prefix=d50 + b"Y")
+    assert r["sum_promo"] == 0 and r["count"] > 0
+    r = oracle.q14(t, *p["q14"][:2], prefix=d50)  # the whole value as the prefix: a match
+    assert r["sum_promo"] > 0
+    db = sqlite_load(t)
+    assert sqlite_q14(db, *p["q14"][:2], prefix=(d50 + b"Y").decode())[1] == 0
+
+
 @pytest.mark.parametrize("seed", [1, 2, 3])
 def test_brute_force_tiny(seed):
     t = mutate(chgen.generate(1, 3, seed=seed, scale=chgen.TINY), seed)
