@@ -318,6 +318,21 @@ def cpu_oracle_sample(w_lo, sample_w, mode):
     return n / dt, dt, n, pc.used
 
 
+def workload_name(a, world):
+    """The `config.workload` string of a run (both arms print the same one)."""
+    qs = "+".join(x.strip().upper() for x in a.plans.split(",") if x.strip())
+    if a.total_warehouses is not None:
+        w = f"CH {qs} per step over W={a.total_warehouses} warehouses split over {world} GPU(s)"
+    else:
+        w = f"CH {qs} per step over W={a.warehouses} warehouses per GPU"
+    return w + f" ('{a.mode}' TPC-C population, seed 1)"
+
+
+def rows_counted(a):
+    qs = " + ".join(x.strip().upper() for x in a.plans.split(",") if x.strip())
+    return f"each visible order_line row counted once per step; one step = CH {qs} over the snapshot"
+
+
 def run_reference(a):
     rank, world, _ = dist_env()
     if rank != 0:
@@ -327,31 +342,35 @@ def run_reference(a):
     sample_w = 10
     t = chgen.generate(1, 1 + sample_w, seed=1, mode=a.mode)
     n = len(t["order_line"]["ol_w_id"])
+    want = [x.strip() for x in a.plans.split(",") if x.strip()]
+    fns = [f for q, f in (("q6", lambda: oracle.q6(t, *Q6_P)), ("q1", lambda: oracle.q1(t, *Q1_P)),
+                          ("q18", lambda: oracle.q18(t, *Q18_P))) if q in want]
     with pinned_core(1) as pc:
         for _ in range(a.warmup):
-            oracle.q6(t, *Q6_P); oracle.q1(t, *Q1_P); oracle.q18(t, *Q18_P)
+            for f in fns:
+                f()
         t0 = time.perf_counter()
         for _ in range(a.steps):
-            oracle.q6(t, *Q6_P); oracle.q1(t, *Q1_P); oracle.q18(t, *Q18_P)
+            for f in fns:
+                f()
         dt = time.perf_counter() - t0
     value = n * a.steps / dt
-    sample = (f"each step = oracle Q6+Q1+Q18 over W={sample_w} warehouses ({n} order_line rows, "
+    sample = (f"each step = oracle {'+'.join(q.upper() for q in want)} over W={sample_w} warehouses ({n} order_line rows, "
               f"'{a.mode}', seed 1), single thread pinned to core {pc.used}")
     print(json.dumps({
         "impl": "reference", "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": a.gpus,
         "steps": a.steps, "warmup": a.warmup, "ms_per_step": dt / a.steps * 1e3,
         "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "int64",
-        "data": "synthetic", "config": {"workload": f"CH Q6+Q1+Q18 per step, sample W={sample_w}",
-                                        "mode": a.mode, "rows_counted": ROWS_COUNTED},
+        "data": "synthetic", "config": {"workload": workload_name(a, a.gpus), "rows_counted": rows_counted(a),
+                                        "reference_sample": f"W={sample_w} of the workload's warehouses per "
+                                                            "step (rows/s is size-independent for the "
+                                                            "row-at-a-time oracle)"},
         "cpu_baseline": dict({"value": value, "unit": UNIT, "cores": 1, "kind": "oracle", "sample": sample,
                               "pinned_core": pc.used}, **host_cpu()),
         "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }))
     return 0
 
-
-ROWS_COUNTED = ("each visible order_line row counted once per step; one step = CH Q6 + Q1 + Q18 "
-                "over the snapshot (all three read every order_line row)")
 
 
 # ----------------------------------------------------------------------- ours --
@@ -786,15 +805,11 @@ def main():
             "ms_per_step_host_return": round(step_host_ms, 5),
             "scaling": "strong" if strong else "weak", "vs_baseline": None, "dtype": "int64",
             "data": "synthetic",
-            "config": {"workload": (f"CH {'+'.join(q.upper() for q in ALL)} per step over W={W} warehouses split over {world} GPU(s)"
-                                    if strong else
-                                    f"CH {'+'.join(q.upper() for q in ALL)} per step over W={a.warehouses} warehouses per GPU")
-                                   + f" ('{a.mode}' TPC-C population, seed 1)",
+            "config": {"workload": workload_name(a, world),
                        "warehouses_total": W, "warehouses_per_gpu": W / world,
                        "order_line_rows_total": rows_total, "order_line_rows_rank0": n_ol,
                        "orders_rows_rank0": n_o, "customer_rows_rank0": n_c,
-                       "rows_counted": ("each visible order_line row counted once per step; one step = CH "
-                                        + " + ".join(q.upper() for q in ALL) + " over the snapshot"),
+                       "rows_counted": rows_counted(a),
                        "queries_per_step": len(ALL),
                        **({"shared_device": "FUNCTIONAL CHECK ONLY: all ranks on one GPU"} if a.share_device else {}), "parallelism": f"row-sharded by warehouse x{world}",
                        "merge": ("peer-memory kernels over NVLink (Q6 allreduce, Q1 group lists, Q18 "
