@@ -657,6 +657,41 @@ def w100():
     return chgen.generate(1, 101, seed=1, mode="spread")
 
 
+def test_bench_line_contract():
+    """bench.py at N=1 on a small snapshot prints one JSON line with every key the measurement
+    contract names, consistent with itself."""
+    import json as _json
+    import os
+    import subprocess
+    import sys
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    env = {k: v for k, v in os.environ.items() if k not in ("RANK", "WORLD_SIZE", "LOCAL_RANK")}
+    r = subprocess.run([sys.executable, os.path.join(root, "bench.py"), "--steps", "3", "--warmup", "3",
+                        "--warehouses", "2", "--e2e-steps", "3", "--inc-neworders", "500",
+                        "--inc-deliveries", "50"], capture_output=True, text=True, env=env, timeout=900)
+    assert r.returncode == 0, r.stderr[-3000:]
+    d = _json.loads([x for x in r.stdout.splitlines() if x.startswith("{")][-1])
+    for k in ("metric", "value", "unit", "n_gpus", "steps", "warmup", "ms_per_step", "higher_is_better",
+              "scaling", "vs_baseline", "dtype", "data", "config", "roofline", "cpu_baseline", "e2e",
+              "gpu_launches", "clocks", "c1", "c2", "c3", "e2e_incremental"):
+        assert k in d, k
+    assert d["n_gpus"] == 1 and d["steps"] == 3 and d["warmup"] == 3 and d["higher_is_better"] is True
+    assert d["value"] > 0 and d["ms_per_step"] > 0 and d["gpu_launches"] > 0
+    assert math.isclose(d["value"], d["config"]["order_line_rows_total"] / (d["ms_per_step"] / 1e3), rel_tol=1e-6)
+    roof = d["roofline"]
+    for k in ("bound", "achieved", "peak", "unit", "frac", "traffic"):
+        assert k in roof, k
+    assert math.isclose(roof["frac"], roof["achieved"] / roof["peak"], rel_tol=1e-3)
+    for k in ("value", "unit", "h2d_bytes_per_step", "d2h_bytes_per_step"):
+        assert k in d["e2e"], k
+    assert d["e2e"]["h2d_bytes_per_step"] > 0 and d["e2e"]["d2h_bytes_per_step"] > 0
+    assert d["e2e"]["value"] < d["value"]  # host copies inside: not the device figure again
+    cb = d["cpu_baseline"]
+    assert cb["kind"] == "oracle" and cb["cores"] == 1 and cb["value"] > 0
+    assert {"sm_mhz", "sm_max_mhz", "reasons"} <= set(d["clocks"])
+    assert d["e2e_incremental"]["h2d_bytes_per_step"] > 0 and d["e2e_incremental"]["pipelined"]["value"] > 0
+
+
 def test_full_size_w100_bench_config(h, w100):
     """BASELINE configs[1]/[2] size (W=100, 30M order_line rows), launched exactly as bench.py
     does (same engine entry points, default CH params), compared element by element."""
