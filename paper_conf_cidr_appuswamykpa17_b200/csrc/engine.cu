@@ -850,13 +850,10 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
     }
     CK(cudaEventRecord(pend.t3, e->copy));
     CK(cudaGetLastError());
-    {   // the statistics to the host by a kernel's stores to the mapped pinned block, not a DMA: a
-        // DMA here would queue behind any large device-to-host copy of the caller's (measured:
-        // a refresh under a concurrent 120 MB result read-back took 2.4 ms instead of ~0.3)
-        void *dst = nullptr;
-        CK(cudaHostGetDevicePointer(&dst, pend.stats_host, 0));
-        launch_copy_words(dst, stats_dev, kStatTotal, e->copy);
-    }
+    // (a DMA, not a kernel's stores to the mapped block: under a saturating query loop a kernel
+    // waits for an SM slot — measured in config C5: refresh 4.8 vs 8.1 ms, lag p99 138 vs 622 ms —
+    // while the DMA only queues behind a caller's own large device-to-host copy)
+    CK(cudaMemcpyAsync(pend.stats_host, stats_dev, kStatTotal, cudaMemcpyDeviceToHost, e->copy));
     CK(cudaEventCreateWithFlags(&pend.done, cudaEventDisableTiming));
     CK(cudaEventRecord(pend.done, e->copy));
     pend.view = v;
@@ -2121,7 +2118,15 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         if (const char *impl = std::getenv("H2TAP_COW")) e->cow_full = std::strcmp(impl, "full") == 0;
 
         CK(cudaStreamCreateWithFlags(&e->compute, cudaStreamNonBlocking));
-        CK(cudaStreamCreateWithFlags(&e->copy, cudaStreamNonBlocking));
+        {   // the refresh stream at the highest priority: its kernels (zone maps, copy-on-write) are
+            // scheduled ahead of queued query blocks as SM slots free up, so a refresh under a
+            // saturating query loop (config C5) does not wait behind whole query kernels
+            // (H2TAP_COPY_PRIORITY=0: default priority, A/B)
+            int lo = 0, hi = 0;
+            CK(cudaDeviceGetStreamPriorityRange(&lo, &hi));
+            const char *cp = std::getenv("H2TAP_COPY_PRIORITY");
+            CK(cudaStreamCreateWithPriority(&e->copy, cudaStreamNonBlocking, (cp && cp[0] == '0') ? lo : hi));
+        }
         CK(cudaStreamCreateWithFlags(&e->side, cudaStreamNonBlocking));
         CK(cudaEventCreateWithFlags(&e->ev_fork, cudaEventDisableTiming));
         CK(cudaEventCreateWithFlags(&e->ev_join, cudaEventDisableTiming));

@@ -354,8 +354,6 @@ void launch_gate(unsigned long long ns, cudaStream_t st);  // profiling only  //
 void launch_minmax_i32(const int32_t *p, uint64_t n, int *out, int num_sms, cudaStream_t st);
 // 64-bit zone map: out[2k] = INT64_MAX, out[2k + 1] = INT64_MIN; then min / max of p[0, n) merged in
 void launch_stats_init64(long long *out, int n_pairs, cudaStream_t st);
-// bytes (a multiple of 8) from device memory to a mapped pinned host address, written by one block
-void launch_copy_words(void *dst_mapped, const void *src, size_t bytes, cudaStream_t st);
 void launch_minmax_i64(const int64_t *p, uint64_t n, long long *out, int num_sms, cudaStream_t st);
 // copy-on-write of updated columns (NEXT-1): page = kCowPageRows rows, one dirty bit per page
 constexpr uint64_t kCowPageRows = 4096;

@@ -25,14 +25,6 @@ __global__ void stats_init_kernel(int *out, int n_pairs) {
     if (i < n_pairs) { out[2 * i] = INT_MAX; out[2 * i + 1] = INT_MIN; }
 }
 
-// A few words device -> pinned host memory written by the SMs (the pointer is the mapped address):
-// the refresh's statistics reach the host without a DMA, so they do not queue behind a large
-// device-to-host copy the caller may have running on a copy engine
-__global__ void copy_words_kernel(unsigned long long *__restrict__ dst, const unsigned long long *__restrict__ src,
-                                  int n) {
-    for (int i = threadIdx.x; i < n; i += blockDim.x) dst[i] = __ldcg(src + i);
-}
-
 __global__ void stats_init64_kernel(long long *out, int n_pairs) {
     const int i = blockIdx.x * blockDim.x + threadIdx.x;
     if (i < n_pairs) { out[2 * i] = INT64_MAX; out[2 * i + 1] = INT64_MIN; }
@@ -190,11 +182,6 @@ void launch_stats_init(int *out, int n_pairs, cudaStream_t st) {
     stats_init_kernel<<<(n_pairs + 127) / 128, 128, 0, st>>>(out, n_pairs);
 }
 
-void launch_copy_words(void *dst_mapped, const void *src, size_t bytes, cudaStream_t st) {
-    copy_words_kernel<<<1, 128, 0, st>>>(static_cast<unsigned long long *>(dst_mapped),
-                                         static_cast<const unsigned long long *>(src), (int)(bytes / 8));
-}
-
 void launch_stats_init64(long long *out, int n_pairs, cudaStream_t st) {
     stats_init64_kernel<<<(n_pairs + 127) / 128, 128, 0, st>>>(out, n_pairs);
 }
@@ -236,8 +223,7 @@ cudaError_t set_attributes_store(int num_sms) {
         (const void *)cow_catchup_kernel<8>,
         (const void *)gate_kernel,
         (const void *)minmax_kernel,
-        (const void *)stats_init_kernel, (const void *)stats_init64_kernel, (const void *)minmax64_kernel,
-        (const void *)copy_words_kernel};
+        (const void *)stats_init_kernel, (const void *)stats_init64_kernel, (const void *)minmax64_kernel};
     const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
     if (le != cudaSuccess) return le;
     return cudaSuccess;
