@@ -662,7 +662,11 @@ def main():
     kavg = {k: float(np.mean(v)) for k, v in kern.items()}
     sort_passes = ("v1" if os.environ.get("H2TAP_ORDER") == "v1"
                    else "v2" if os.environ.get("H2TAP_ORDER_CARRY") == "0" else "carry")
-    dominant = max(kavg, key=kavg.get) if kavg else None
+    # the dominant kernel: the largest share of the step among the kernels with a byte model (at
+    # W = 100 the shared scan; on tiny snapshots a launch-bound kernel could otherwise win)
+    modeled = [k for k in kavg if alg_bytes(k, n_ol, n_o, n_c, n_pass, sort_passes, box if plan_dense else None,
+                                            plan_clustered and sort_passes == "carry")]
+    dominant = max(modeled, key=kavg.get) if modeled else None
     peak, peak_src = peaks()
     rpeak = read_stream_peak(h, eng, stream) if rank == 0 else None
     roof = None

@@ -406,6 +406,8 @@ struct h2tap_engine {
     FreeOrder free_order;
     cudaEvent_t q_begin = nullptr, q_end = nullptr;
     cudaEvent_t b_begin = nullptr, b_end = nullptr;  // the last h2tap_run_queries batch on the device
+    unsigned long long *pages_dev = nullptr;  // copy-on-write pages copied so far (device counter,
+                                              // read by h2tap_get_store_stats only)
     float last_batch_ms = -1.f;
 
     std::mutex load_mu, query_mu, view_mu, pend_mu;
@@ -476,9 +478,6 @@ void publish_ready(h2tap_engine *e, bool wait) {
             S.rows_appended += p.rows_appended;
             S.rows_updated += p.rows_updated;
             S.cow_full_copies += p.full_copies;
-            uint64_t pages;
-            std::memcpy(&pages, reinterpret_cast<char *>(p.stats_host) + kStatBytes, 8);
-            S.cow_pages_copied += pages;
             float a = 0, b = 0;
             CK(cudaEventElapsedTime(&a, p.t0, p.t1));
             CK(cudaEventElapsedTime(&b, p.t1, p.t2));
@@ -556,6 +555,26 @@ bool h2d(h2tap_engine *e, void *dst, const void *src, size_t bytes) {
         CK(cudaEventRecord(S.ev[k], e->copy));
     }
     return false;
+}
+
+// Zone-map deltas of a small refresh on the host, over the caller's own buffers (appended rows,
+// update values): no device kernel and no device-to-host copy on the refresh's critical path — a
+// kernel there waits for an SM slot under a saturating query loop, a DMA behind any large
+// read-back of the caller's. Large deltas (full reloads) keep the device kernels.
+constexpr uint64_t kHostStatsValues = 8u << 20;  // values scanned on the host at most per refresh
+__attribute__((target_clones("avx2", "default")))
+void host_minmax_i32(const int32_t *p, uint64_t n, int &mn, int &mx) {
+    int a = INT32_MAX, b = INT32_MIN;
+    for (uint64_t i = 0; i < n; ++i) { a = p[i] < a ? p[i] : a; b = p[i] > b ? p[i] : b; }
+    mn = std::min(mn, a);
+    mx = std::max(mx, b);
+}
+__attribute__((target_clones("avx2", "default")))
+void host_minmax_i64(const int64_t *p, uint64_t n, long long &mn, long long &mx) {
+    long long a = INT64_MAX, b = INT64_MIN;
+    for (uint64_t i = 0; i < n; ++i) { a = p[i] < a ? p[i] : a; b = p[i] > b ? p[i] : b; }
+    mn = std::min(mn, a);
+    mx = std::max(mx, b);
 }
 
 h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntables,
@@ -687,12 +706,29 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
     pend.stats_host = static_cast<int *>(pend.stats_block.first);
     int *stats_dev = static_cast<int *>(e->load_arena.get("load.stats", kStatTotal));
     auto *stats64_dev = reinterpret_cast<long long *>(reinterpret_cast<char *>(stats_dev) + kStat64Off);
-    auto *pages_dev = reinterpret_cast<unsigned long long *>(reinterpret_cast<char *>(stats_dev) + kStatBytes);
+    unsigned long long *pages_dev = e->pages_dev;
+    // zone maps on the host when the delta is small (see host_minmax_i32)
+    bool host_stats;
+    {
+        uint64_t vals = 0;
+        for (uint32_t i = 0; i < ntables; ++i) {
+            const h2tap_table &t = tables[i];
+            vals += (t.row_count - t.first_row) * (uint64_t)(stat_cols(t.table_id) + 1);
+        }
+        for (uint32_t i = 0; i < nupdates; ++i) vals += updates[i].n;
+        host_stats = vals <= kHostStatsValues || (flags & H2TAP_LOAD_ZERO_COPY);
+    }
+    int *stats_h = pend.stats_host;
+    long long *stats64_h = reinterpret_cast<long long *>(reinterpret_cast<char *>(stats_h) + kStat64Off);
     for (cudaEvent_t *ev : {&pend.t0, &pend.t1, &pend.t2, &pend.t3}) CK(cudaEventCreate(ev));
     CK(cudaEventRecord(pend.t0, e->copy));
-    launch_stats_init(stats_dev, kTables * kStatCols, e->copy);
-    launch_stats_init64(stats64_dev, kTables, e->copy);
-    CK(cudaMemsetAsync(pages_dev, 0, 8, e->copy));
+    if (host_stats) {
+        for (int i = 0; i < kTables * kStatCols; ++i) { stats_h[2 * i] = INT32_MAX; stats_h[2 * i + 1] = INT32_MIN; }
+        for (int i = 0; i < kTables; ++i) { stats64_h[2 * i] = INT64_MAX; stats64_h[2 * i + 1] = INT64_MIN; }
+    } else {
+        launch_stats_init(stats_dev, kTables * kStatCols, e->copy);
+        launch_stats_init64(stats64_dev, kTables, e->copy);
+    }
     for (uint32_t i = 0; i < ntables; ++i) {
         const h2tap_table &t = tables[i];
         TableState &ts = e->tables[t.table_id];
@@ -768,17 +804,38 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
         v->n[t.table_id] = t.row_count;
         pend.loaded[t.table_id] = true;
         pend.full[t.table_id] = full;
-        // zone map of the appended rows' key columns, on the copy stream after their H2D
+        // zone map of the appended rows' key columns: on the host from the caller's buffers (small
+        // deltas), else on the copy stream after their H2D
+        auto host_col = [&](int cid) -> const void * {
+            for (uint32_t c = 0; c < t.ncols; ++c)
+                if ((int)t.cols[c].column_id == cid) return t.cols[c].host_data;
+            return nullptr;
+        };
+        const uint64_t nrows_delta = t.row_count - t.first_row;
         if (const int c64 = stat64_col(t.table_id); c64 >= 0 && v->col[t.table_id][c64] && !v->host[t.table_id][c64]) {
-            launch_minmax_i64(static_cast<const int64_t *>(v->col[t.table_id][c64]) + t.first_row,
-                              t.row_count - t.first_row, stats64_dev + 2 * t.table_id, e->num_sms, e->copy);
+            if (host_stats) {
+                if (const void *hp = host_col(c64))
+                    host_minmax_i64(static_cast<const int64_t *>(hp), nrows_delta, stats64_h[2 * t.table_id],
+                                    stats64_h[2 * t.table_id + 1]);
+            } else {
+                launch_minmax_i64(static_cast<const int64_t *>(v->col[t.table_id][c64]) + t.first_row,
+                                  nrows_delta, stats64_dev + 2 * t.table_id, e->num_sms, e->copy);
+            }
             pend.stats64_ok[t.table_id] = true;
         }
-        for (int c = 0; c < stat_cols(t.table_id); ++c)
-            if (stat_col(t.table_id, c) >= 0 && v->col[t.table_id][stat_col(t.table_id, c)])
-                launch_minmax_i32(static_cast<const int32_t *>(v->col[t.table_id][stat_col(t.table_id, c)]) + t.first_row,
-                                  t.row_count - t.first_row,
+        for (int c = 0; c < stat_cols(t.table_id); ++c) {
+            const int cid = stat_col(t.table_id, c);
+            if (cid < 0 || !v->col[t.table_id][cid]) continue;
+            if (host_stats) {
+                if (const void *hp = host_col(cid))
+                    host_minmax_i32(static_cast<const int32_t *>(hp), nrows_delta,
+                                    stats_h[(t.table_id * kStatCols + c) * 2],
+                                    stats_h[(t.table_id * kStatCols + c) * 2 + 1]);
+            } else {
+                launch_minmax_i32(static_cast<const int32_t *>(v->col[t.table_id][cid]) + t.first_row, nrows_delta,
                                   stats_dev + (t.table_id * kStatCols + c) * 2, e->num_sms, e->copy);
+            }
+        }
     }
     CK(cudaEventRecord(pend.t1, e->copy));
     // ---- in-place updates: upload every update's row ids and values first (one arena region;
@@ -831,13 +888,23 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
             const auto *rows_d = reinterpret_cast<const uint32_t *>(upd_dev + upd_off[i]);
             const void *vals_d = upd_dev + upd_off[i] + round_up16(u.n * 4);
             launch_apply_updates(cs.alt->ptr, (uint32_t)es, next_bits, rows_d, vals_d, u.n, e->num_sms, e->copy);
-            if ((int)u.column_id == stat64_col(u.table_id))  // 64-bit zone map: widen
-                launch_minmax_i64(static_cast<const int64_t *>(vals_d), u.n, stats64_dev + 2 * u.table_id,
-                                  e->num_sms, e->copy);
-            if (stat_slot(u.table_id, u.column_id) >= 0)  // zone map: widen
-                launch_minmax_i32(static_cast<const int32_t *>(vals_d), u.n,
-                                  stats_dev + (u.table_id * kStatCols + stat_slot(u.table_id, u.column_id)) * 2,
-                                  e->num_sms, e->copy);
+            if ((int)u.column_id == stat64_col(u.table_id)) {  // 64-bit zone map: widen
+                if (host_stats)
+                    host_minmax_i64(static_cast<const int64_t *>(u.values), u.n, stats64_h[2 * u.table_id],
+                                    stats64_h[2 * u.table_id + 1]);
+                else
+                    launch_minmax_i64(static_cast<const int64_t *>(vals_d), u.n, stats64_dev + 2 * u.table_id,
+                                      e->num_sms, e->copy);
+            }
+            if (const int sl = stat_slot(u.table_id, u.column_id); sl >= 0) {  // zone map: widen
+                if (host_stats)
+                    host_minmax_i32(static_cast<const int32_t *>(u.values), u.n,
+                                    stats_h[(u.table_id * kStatCols + sl) * 2],
+                                    stats_h[(u.table_id * kStatCols + sl) * 2 + 1]);
+                else
+                    launch_minmax_i32(static_cast<const int32_t *>(vals_d), u.n,
+                                      stats_dev + (u.table_id * kStatCols + sl) * 2, e->num_sms, e->copy);
+            }
         }
         std::swap(cs.cur, cs.alt);
         std::swap(cs.bits, cs.bits_next);
@@ -850,10 +917,10 @@ h2tap_status load_impl(h2tap_engine *e, const h2tap_table *tables, uint32_t ntab
     }
     CK(cudaEventRecord(pend.t3, e->copy));
     CK(cudaGetLastError());
-    // (a DMA, not a kernel's stores to the mapped block: under a saturating query loop a kernel
-    // waits for an SM slot — measured in config C5: refresh 4.8 vs 8.1 ms, lag p99 138 vs 622 ms —
-    // while the DMA only queues behind a caller's own large device-to-host copy)
-    CK(cudaMemcpyAsync(pend.stats_host, stats_dev, kStatTotal, cudaMemcpyDeviceToHost, e->copy));
+    // device statistics (large deltas): one DMA, not a kernel's stores to the mapped block (under a
+    // saturating query loop a kernel waits for an SM slot — config C5: refresh 4.8 vs 8.1 ms, lag
+    // p99 138 vs 622 ms)
+    if (!host_stats) CK(cudaMemcpyAsync(pend.stats_host, stats_dev, kStatTotal, cudaMemcpyDeviceToHost, e->copy));
     CK(cudaEventCreateWithFlags(&pend.done, cudaEventDisableTiming));
     CK(cudaEventRecord(pend.done, e->copy));
     pend.view = v;
@@ -2133,6 +2200,8 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         if (const char *q = std::getenv("H2TAP_Q18_STREAM")) e->q18_side = std::atoi(q) != 0;
         if (const char *q = std::getenv("H2TAP_Q1_SIDE")) e->q1_side = std::atoi(q) != 0;
         CK(cudaStreamCreateWithFlags(&e->reaper, cudaStreamNonBlocking));
+        CK(cudaMalloc(&e->pages_dev, 8));
+        CK(cudaMemset(e->pages_dev, 0, 8));
         e->free_order = FreeOrder{e->compute, e->copy, e->reaper};
         {   // keep freed pool memory cached (no release to the OS at stream syncs)
             cudaMemPool_t pool;
@@ -2230,6 +2299,12 @@ h2tap_status h2tap_get_store_stats(h2tap_engine *e, h2tap_store_stats *out) {
         {
             std::lock_guard<std::mutex> gp(e->pend_mu);
             *out = e->sstats;
+        }
+        {   // the copy-on-write page counter lives on the device (no copy per refresh); the copies of
+            // the refreshes published so far are complete (publish waited for their events)
+            unsigned long long pages = 0;
+            CK(cudaMemcpy(&pages, e->pages_dev, 8, cudaMemcpyDeviceToHost));
+            out->cow_pages_copied = pages;
         }
         uint64_t bytes = 0;
         for (auto &t : e->tables)
@@ -2426,6 +2501,7 @@ void h2tap_close(h2tap_engine *e) {
     cudaStreamSynchronize(e->copy);
     for (void *p : e->peer.opened) cudaIpcCloseMemHandle(p);
     if (e->peer.seg) cudaFree(e->peer.seg);
+    if (e->pages_dev) cudaFree(e->pages_dev);
     if (e->peer.err_host) cudaFreeHost(e->peer.err_host);
     for (auto &p : e->pending) {
         for (cudaEvent_t ev : {p.done, p.t0, p.t1, p.t2, p.t3}) cudaEventDestroy(ev);
