@@ -15,6 +15,7 @@
 // 64-bit atomic per block. The same kernels read HBM or mapped pinned host memory (UVA, the
 // paper's Caldera mechanism, L484-490, L568-572): only the pointer differs.
 #include <cstdint>
+#include <cstdlib>
 #include <cuda_runtime.h>
 
 #include "kernels.cuh"
@@ -138,6 +139,86 @@ pax_sum_kernel(const int32_t *__restrict__ data, uint64_t n, int log_ncols, int 
     block_add(acc, out);
 }
 
+// PAX with N (selected attributes) a power of two — the paper's N = 1, 2, 4, 8, 16: the selected
+// minipages of page p form V = N x vpm consecutive 16-byte vectors of one stream, and a warp
+// iteration takes 128 consecutive stream vectors (4 per lane, all loads in flight first). With V
+// and 128 both powers of two every lane's (page offset, minipage, vector) decomposition is either
+// the same for every iteration (V <= 128) or shifts by a whole number of minipages (V > 128), so
+// the loop does no divisions and little address arithmetic (the general kernel above spent its
+// issue slots there: 0.6 of the copy peak at N = 16 where the stream is the whole table).
+#ifndef PAX_U
+#define PAX_U 4
+#endif
+constexpr int kPaxU = PAX_U;
+__global__ void __launch_bounds__(kThreads)
+pax_pow2_sum_kernel(const int32_t *__restrict__ data, uint64_t n, int log_ncols, int log_mp, int log_n,
+                    LayoutSel sel, unsigned long long *out) {
+    __shared__ int cols[kMaxLayoutSel];
+    for (int i = threadIdx.x; i < sel.n; i += kThreads) cols[i] = sel.col[i];
+    __syncthreads();
+    const int lane = threadIdx.x & 31;
+    const int log_vpm = log_mp - 2, log_v = log_n + log_vpm;  // vectors per minipage / per page
+    const uint64_t pages = (n + (1ull << log_mp) - 1) >> log_mp;
+    const uint64_t total = pages << log_v;                     // stream vectors
+    const uint64_t gwarp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
+    constexpr int kW = 32 * kPaxU;                              // stream vectors per warp iteration
+    const unsigned vmask = (1u << log_vpm) - 1u;
+    // this lane's k-th vector of an iteration, o = k * 32 + lane: with V = 2^log_v <= kW the
+    // iteration starts on a page boundary and o decomposes into a fixed (page offset, minipage
+    // column, vector) — precomputed; with V > kW the minipage shifts by a fixed amount per step
+    const bool small_v = log_v <= __ffs(kW) - 1;
+    unsigned dpage[kPaxU], colv[kPaxU];                         // colv = (column << 16) | vector
+#pragma unroll
+    for (int u = 0; u < kPaxU; ++u) {
+        const unsigned o = (unsigned)u * 32 + lane;
+        const unsigned within = small_v ? (o & ((1u << log_v) - 1u)) : o;
+        dpage[u] = small_v ? (o >> log_v) : 0u;
+        colv[u] = small_v ? (((unsigned)cols[within >> log_vpm] << 16) | (within & vmask)) : 0u;
+    }
+    long long acc = 0;
+    const uint64_t full = (n >> log_mp) << log_v;  // stream vectors of the complete pages
+    for (uint64_t q0 = gwarp * kW; q0 < total; q0 += nwarps * kW) {
+        const uint64_t p0 = q0 >> log_v;
+        const unsigned j0 = small_v ? 0u : (unsigned)((q0 & ((1ull << log_v) - 1)) >> log_vpm);
+        if (q0 + kW <= full) {  // whole pages only (all but the last iterations): no row masks
+            int4 x[kPaxU];
+#pragma unroll
+            for (int u = 0; u < kPaxU; ++u) {
+                const unsigned o = (unsigned)u * 32 + lane;
+                uint64_t p;
+                unsigned col, v;
+                if (small_v) { p = p0 + dpage[u]; col = colv[u] >> 16; v = colv[u] & 0xffffu; }
+                else { p = p0; col = (unsigned)cols[j0 + (o >> log_vpm)]; v = o & vmask; }
+                x[u] = ld_stream(reinterpret_cast<const int4 *>(data + ((((p << log_ncols) + col) << log_mp) + 4 * (uint64_t)v)));
+            }
+#pragma unroll
+            for (int u = 0; u < kPaxU; ++u) acc += (long long)x[u].x + x[u].y + x[u].z + x[u].w;
+            continue;
+        }
+        int4 x[kPaxU];
+        unsigned sel4[kPaxU];
+#pragma unroll
+        for (int u = 0; u < kPaxU; ++u) {
+            const unsigned o = (unsigned)u * 32 + lane;
+            uint64_t p;
+            unsigned col, v;
+            if (small_v) { p = p0 + dpage[u]; col = colv[u] >> 16; v = colv[u] & 0xffffu; }
+            else { p = p0; col = (unsigned)cols[j0 + (o >> log_vpm)]; v = o & vmask; }
+            const uint64_t row0 = (p << log_mp) + 4 * (uint64_t)v;
+            sel4[u] = (q0 + o >= total || row0 >= n) ? 0u : (n - row0 >= 4 ? 0xfu : (1u << (unsigned)(n - row0)) - 1u);
+            if (sel4[u]) {
+                const uint64_t off = (((p << log_ncols) + col) << log_mp) + 4 * (uint64_t)v;
+                x[u] = ld_stream(reinterpret_cast<const int4 *>(data + off));
+            }
+        }
+#pragma unroll
+        for (int u = 0; u < kPaxU; ++u)
+            if (sel4[u]) acc += lanes_sum(x[u], sel4[u]);
+    }
+    block_add(acc, out);
+}
+
 // NSM: records of 2^log_ncols attributes (>= 4) back to back; vector e holds attributes
 // (4e mod ncols) .. +3 of record 4e / ncols. Vectors without a selected attribute are not loaded.
 __global__ void __launch_bounds__(kThreads)
@@ -182,8 +263,16 @@ void launch_layout_sum(const int32_t *data, int layout, uint64_t n, int log_ncol
     } else if (layout == kLayoutPax) {
         const uint64_t pages = (n + (1ull << log_mp) - 1) >> log_mp;
         const uint64_t vpm = 1ull << (log_mp - 2);
-        pax_sum_kernel<<<grid_for(pages * sel.n * vpm / kUnroll, num_sms), kThreads, 0, st>>>(
-            data, n, log_ncols, log_mp, sel, out);
+        static const bool general = [] { const char *v = std::getenv("H2TAP_PAX_GENERAL"); return v && v[0] == '1'; }();
+        if (!general && (sel.n & (sel.n - 1)) == 0) {  // N a power of two
+            int log_n = 0;
+            while ((1 << log_n) < sel.n) ++log_n;
+            pax_pow2_sum_kernel<<<grid_for(pages * sel.n * vpm / kPaxU, num_sms), kThreads, 0, st>>>(
+                data, n, log_ncols, log_mp, log_n, sel, out);
+        } else {
+            pax_sum_kernel<<<grid_for(pages * sel.n * vpm / kUnroll, num_sms), kThreads, 0, st>>>(
+                data, n, log_ncols, log_mp, sel, out);
+        }
     } else {
         nsm_sum_kernel<<<grid_for(((n << log_ncols) >> 2) / kUnroll, num_sms), kThreads, 0, st>>>(
             data, n, log_ncols, mask, out);
@@ -208,7 +297,8 @@ cudaError_t set_attributes_layout(int num_sms) {
     static const void *const kKernels[] = {
         (const void *)dsm_sum_kernel,
         (const void *)nsm_sum_kernel,
-        (const void *)pax_sum_kernel};
+        (const void *)pax_sum_kernel,
+        (const void *)pax_pow2_sum_kernel};
     const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
     if (le != cudaSuccess) return le;
     return cudaSuccess;
