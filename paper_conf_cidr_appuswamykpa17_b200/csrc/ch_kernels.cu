@@ -214,7 +214,23 @@ __global__ void sg_peer_merge_kernel(PeerArgs p, SmallGroups g) {
 }
 
 // ========================================================= orders index ==
+// Clustered orders (as for Q18): count the rows not at their own dense slot; 0 =
+// the index is the identity and nothing is cleared or built. Resets the next query's counter.
+__global__ void jx_verify_kernel(JoinIndex j, const int32_t *__restrict__ w, const int32_t *__restrict__ d,
+                                 const int32_t *__restrict__ id, uint64_t n) {
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    const uint64_t n_pad = (n + 31) & ~31ull;
+    for (uint64_t r = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; r < n_pad; r += stride) {
+        unsigned long long s = 0;
+        const bool bad = r < n && (!dense_slot(j, __ldcs(w + r), __ldcs(d + r), __ldcs(id + r), s) || s != r);
+        const unsigned int b = __ballot_sync(kFull, bad);
+        if (b && (threadIdx.x & 31) == __ffs(b) - 1) atomicAdd(j.viol, 1u);
+    }
+    if (blockIdx.x == 0 && threadIdx.x == 0 && j.viol_next) *j.viol_next = 0u;
+}
+
 __global__ void jx_clear_kernel(JoinIndex j) {
+    if (jx_identity(j)) return;  // positional: the slots are never read
     const uint64_t words = jx_words(j);
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < words;
          i += (uint64_t)gridDim.x * blockDim.x)
@@ -224,10 +240,12 @@ __global__ void jx_clear_kernel(JoinIndex j) {
 __global__ void jx_build_orders_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
                                        const int32_t *__restrict__ o_id, uint64_t n, JoinIndex j,
                                        unsigned int *err, uint8_t *mark) {
+    const bool ident = jx_identity(j);
+    if (ident && !mark) return;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
          i += (uint64_t)gridDim.x * blockDim.x) {
         if (mark) mark[i] = 0;
-        if (!jx_insert(j, o_w[i], o_d[i], o_id[i], (unsigned int)i, err, kErrDupOrders))
+        if (!ident && !jx_insert(j, o_w[i], o_d[i], o_id[i], (unsigned int)i, err, kErrDupOrders))
             atomicOr(err, kErrDomain);
     }
 }
@@ -473,6 +491,10 @@ void launch_sg_peer_merge(const PeerArgs &p, const SmallGroups &g, cudaStream_t 
 void launch_jx_build_orders(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, uint64_t n_o,
                             const JoinIndex &jo, unsigned int *err, uint8_t *mark, int num_sms,
                             cudaStream_t st) {
+    if (jo.may_ident) {
+        jx_verify_kernel<<<grid_for(n_o, 256, num_sms, 8), 256, 0, st>>>(jo, o_w, o_d, o_id, n_o);
+        count_launches(1);
+    }
     jx_clear_kernel<<<grid_for(jx_words(jo), 256, num_sms, 8), 256, 0, st>>>(jo);
     if (n_o) jx_build_orders_kernel<<<grid_for(n_o, 256, num_sms, 8), 256, 0, st>>>(o_w, o_d, o_id, n_o, jo, err, mark);
     count_launches(n_o ? 2 : 1);
@@ -553,6 +575,7 @@ cudaError_t set_attributes_ch(int num_sms) {
         (const void *)item_map_kernel,
         (const void *)jx_build_orders_kernel,
         (const void *)jx_clear_kernel,
+        (const void *)jx_verify_kernel,
         (const void *)q12_probe_kernel,
         (const void *)q14_finalize_kernel,
         (const void *)q14_kernel<false>,

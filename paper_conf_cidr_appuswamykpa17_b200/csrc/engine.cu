@@ -409,6 +409,7 @@ struct h2tap_engine {
     unsigned long long *pages_dev = nullptr;  // copy-on-write pages copied so far (device counter,
                                               // read by h2tap_get_store_stats only)
     float last_batch_ms = -1.f;
+    uint64_t ch_runs = 0;  // parity of the Q12 / Q4 clustered-index counters
 
     std::mutex load_mu, query_mu, view_mu, pend_mu;
     TableState tables[kTables];
@@ -1806,6 +1807,15 @@ JoinIndex plan_orders_index(h2tap_engine *e, const View &v, QueryCtx &q, const c
     const int O = H2TAP_T_ORDERS;
     JoinIndex jo = plan_index(e, v, O, q.flags & H2TAP_QUERY_HASH_JOIN, "ch.jo");
     q.r->plan_flags = jo.dense ? 1u : 0u;
+    {   // clustered orders (row == dense slot), verified on the device before the build: the
+        // index is then positional and nothing is cleared or inserted
+        auto *viol = static_cast<unsigned int *>(e->arena.get("ch.viol", 64, true, e->compute));
+        const int par = (int)(e->ch_runs++ & 1);
+        static const bool on = [] { const char *x = std::getenv("H2TAP_CLUSTERED"); return !(x && x[0] == '0'); }();
+        jo.may_ident = on && jo.dense && jo.range == v.n[O];
+        jo.viol = viol + par;
+        jo.viol_next = viol + (par ^ 1);
+    }
     (void)plan;
     return jo;
 }

@@ -86,6 +86,22 @@ def run_all(h, L, t, rng=None, n_rand=2):
         assert_groups(L.q(h.H2TAP_Q4, [lo, hi]), oracle.q4(t, lo, hi))
 
 
+@pytest.mark.parametrize("layout", ["clustered", "one_row_swapped", "shuffled"])
+def test_clustered_orders_index_q12_q4(h, L, layout):
+    """Q12 / Q4 take the positional orders index only while the device finds every orders row at
+    its own key slot: the generated table (key order), one swapped pair of rows,
+    fully shuffled rows — all equal the oracle on both index plans."""
+    t = mutate(chgen.generate(1, 3, seed=43), 43)
+    o = t["orders"]
+    perm = np.arange(len(o["o_id"]))
+    if layout == "one_row_swapped":
+        perm[[7, 15000]] = perm[[15000, 7]]
+    elif layout == "shuffled":
+        perm = np.random.default_rng(43).permutation(len(perm))
+    t["orders"] = {k: v[perm].copy() for k, v in o.items()}
+    run_all(h, L, t, np.random.default_rng(43), n_rand=1)
+
+
 def test_golden_fixture(h, L):
     t, p, want = golden_next2()
     L.load(t)
