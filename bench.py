@@ -215,6 +215,9 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None, clustered=F
     the keys and zeroes the accumulators, nothing is built, no slot is read."""
     if clustered:
         return {"q61_shared_scan": 24 * n_ol, "q6_scan_filter_sum": 20 * n_ol, "q1_scan_filter_groupby": 24 * n_ol,
+                # the batch's full pass: Q1's 4 columns + Q18's 3 keys once, the probe's
+                # accumulator read + write per order (DESIGN.md §4.5)
+                "q6118_full_pass": 36 * n_ol + 16 * n_o + 16 * n_o,
                 "q18_init": 12 * (n_o + n_c) + 16 * n_o,            # verify: keys in, acc zeroed
                 "q18_probe_groupjoin": 20 * n_ol + 16 * n_o + 16 * n_o,
                 # one GPU: o_entry_d's bounds come from the snapshot's zone map, acc[] alone is read
@@ -233,6 +236,8 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None, clustered=F
         "q1_scan_filter_groupby": 24 * n_ol,
         # shared scan of the batch's Q6 and Q1: Q1's 4 columns once, both queries
         "q61_shared_scan": 24 * n_ol,
+        # full pass: + Q18's keys; per order one index slot and the accumulator read + write
+        "q6118_full_pass": 36 * n_ol + slot_b * n_o + 16 * n_o + 16 * n_o,
         "q18_init": slot_b * (slots_o + slots_c),               # empty the join indexes
         # keys in, accumulators zeroed, one slot written per build row
         "q18_build": 12 * n_o + 12 * n_c + 16 * n_o + slot_b * (n_o + n_c),

@@ -32,6 +32,16 @@ __device__ __forceinline__ void mbar_wait(uint64_t *bar, unsigned parity) {
         "@!p bra WAIT_%=;\n}"
         :: "r"(smem_u32(bar)), "r"(parity) : "memory");
 }
+// the same with a suspend-time hint (ns): the waiting warp is parked instead of re-issuing
+// try_wait, leaving issue slots to the block's other warps
+__device__ __forceinline__ void mbar_wait_hint(uint64_t *bar, unsigned parity, unsigned ns) {
+    asm volatile(
+        "{\n\t.reg .pred p;\n"
+        "WAIT_%=:\n\t"
+        "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1, %2;\n\t"
+        "@!p bra WAIT_%=;\n}"
+        :: "r"(smem_u32(bar)), "r"(parity), "r"(ns) : "memory");
+}
 // global -> shared bulk copy (size and addresses multiples of 16 B), completion on `bar`, with
 // an L2 evict_first policy (each byte of a scan is read once)
 __device__ __forceinline__ void bulk_g2s(void *dst, const void *src, unsigned bytes, uint64_t *bar,

@@ -381,6 +381,7 @@ struct h2tap_engine {
     bool zc_tma = true;
     int having_unroll = 2;  // H2TAP_HAVING_UNROLL (2 or 4): orders rows per thread in the HAVING pass
     bool shared_scan = true;  // H2TAP_SHARED_SCAN=0: separate Q6 and Q1 scans in a batch (A/B)
+    bool full_pass = true;    // H2TAP_FULL_PASS=0: Q18's probe not in the batch's shared scan (A/B)
     // in-place updates copy only the dirty pages into the shadow (H2TAP_COW=full: always copy the
     // whole column — the A/B baseline of scripts/cow_bench.py)
     bool cow_full = false;
@@ -1002,6 +1003,9 @@ struct QueryCtx {
     int64_t shared_cutoff = 0;              // the paired Q1's cutoff (shared_scan == 1)
     int shared_scan = 0;                    // 1: this Q6 runs the batch's shared Q6+Q1 scan;
                                             // 2: this Q1's scan was done by it
+    QueryCtx *full18 = nullptr;             // (Q6, shared_scan == 1) the batch's Q18 whose probe
+                                            // runs in the same pass (the full pass, §4.5)
+    bool probe_done = false;                // (Q18) init, build and probe ran in the full pass
     const Q18Row *rows = nullptr;
     const long long *amt = nullptr;
     const unsigned int *perm = nullptr;
@@ -1043,6 +1047,8 @@ void give_blocks_to_result(QueryCtx &q) {
 // ---- Q6 (a2 + a7)
 void q1_tables(h2tap_engine *e, Q1Scratch &s);
 
+void q18_pre_probe(h2tap_engine *e, const View &v, QueryCtx &q);
+
 void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
     const int T = H2TAP_T_ORDER_LINE;
     need_cols(v, T, {H2TAP_OL_DELIVERY_D, H2TAP_OL_QUANTITY, H2TAP_OL_AMOUNT}, "Q6");
@@ -1057,7 +1063,21 @@ void launch_q6_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
                          : static_cast<long long *>(dev_block(e, q, 16));
     s.host_out = e->world > 1 ? nullptr : static_cast<long long *>(q.small_dev);
     q.q6_out = s.out;
-    if (q.shared_scan == 1) {  // one pass for this Q6 and the batch's Q1 (its tables filled here)
+    if (q.shared_scan == 1 && q.full18) {  // one pass for this Q6, the batch's Q1 and Q18's probe
+        Q1Scratch t{};
+        q1_tables(e, t);
+        QueryCtx &q18 = *q.full18;
+        q18_pre_probe(e, v, q18);  // the join indexes (and zeroed accumulators) the probe needs
+        e->prof.run("q6118_full_pass", [&] {
+            launch_q6118_tma(colp<int32_t>(v, T, H2TAP_OL_NUMBER), colp<int64_t>(v, T, H2TAP_OL_DELIVERY_D),
+                             colp<int32_t>(v, T, H2TAP_OL_QUANTITY), colp<int64_t>(v, T, H2TAP_OL_AMOUNT),
+                             colp<int32_t>(v, T, H2TAP_OL_W_ID), colp<int32_t>(v, T, H2TAP_OL_D_ID),
+                             colp<int32_t>(v, T, H2TAP_OL_O_ID), v.n[T], q.shared_cutoff, t, q.p[0], q.p[1],
+                             q.p[2], q.p[3], s, q18.q18, e->num_sms, e->compute);
+            CK(cudaGetLastError());
+        });
+        q18.probe_done = true;
+    } else if (q.shared_scan == 1) {  // one pass for this Q6 and the batch's Q1 (its tables filled here)
         Q1Scratch t{};
         q1_tables(e, t);
         e->prof.run("q61_shared_scan", [&] {
@@ -1463,15 +1483,15 @@ void q18_rerun_v2(h2tap_engine *e, QueryCtx &q) {
     sync_compute(e);
 }
 
-void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
-    const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
-    need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}, "Q18");
+// Q18's steps before its probe: join-index plan, init (+ clustered-side verify, zeroed
+// accumulators) and build. Run by the batch's full pass ahead of it, or by launch_q18_plan.
+void q18_pre_probe(h2tap_engine *e, const View &v, QueryCtx &q) {
+    const int O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
     need_cols(v, O, {H2TAP_O_W_ID, H2TAP_O_D_ID, H2TAP_O_ID, H2TAP_O_C_ID, H2TAP_O_OL_CNT, H2TAP_O_ENTRY_D}, "Q18");
     need_cols(v, C, {H2TAP_C_W_ID, H2TAP_C_D_ID, H2TAP_C_ID, H2TAP_C_LAST}, "Q18");
-    const uint64_t n_ol = v.n[OL], n_o = v.n[O], n_c = v.n[C];
+    const uint64_t n_o = v.n[O], n_c = v.n[C];
     q18_scratch(e, v, q, n_o);
     Q18Scratch &s = q.q18;
-
     e->prof.run("q18_init", [&] {
         launch_q18_init(s, colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID),
                         colp<int32_t>(v, O, H2TAP_O_ID), n_o, colp<int32_t>(v, C, H2TAP_C_W_ID),
@@ -1484,13 +1504,25 @@ void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
                          colp<int32_t>(v, C, H2TAP_C_D_ID), colp<int32_t>(v, C, H2TAP_C_ID), n_c, s,
                          e->num_sms, e->compute);
     });
-    e->prof.run("q18_probe_groupjoin", [&] {
-        if (n_ol)
-            ((e->probe_tma || e->zc_tma) && (e->probe_tma || v.any_host(OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}))
-                 ? launch_q18_probe_tma : launch_q18_probe)(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
-                             colp<int32_t>(v, OL, H2TAP_OL_O_ID), colp<int64_t>(v, OL, H2TAP_OL_AMOUNT),
-                             n_ol, s, e->num_sms, e->compute);
-    });
+}
+
+void launch_q18_plan(h2tap_engine *e, const View &v, QueryCtx &q) {
+    const int OL = H2TAP_T_ORDER_LINE, O = H2TAP_T_ORDERS, C = H2TAP_T_CUSTOMER;
+    need_cols(v, OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}, "Q18");
+    need_cols(v, O, {H2TAP_O_W_ID, H2TAP_O_D_ID, H2TAP_O_ID, H2TAP_O_C_ID, H2TAP_O_OL_CNT, H2TAP_O_ENTRY_D}, "Q18");
+    need_cols(v, C, {H2TAP_C_W_ID, H2TAP_C_D_ID, H2TAP_C_ID, H2TAP_C_LAST}, "Q18");
+    const uint64_t n_ol = v.n[OL], n_o = v.n[O];
+    Q18Scratch &s = q.q18;
+    if (!q.probe_done) {  // else the batch's full pass ran them (launch_q6_plan)
+        q18_pre_probe(e, v, q);
+        e->prof.run("q18_probe_groupjoin", [&] {
+            if (n_ol)
+                ((e->probe_tma || e->zc_tma) && (e->probe_tma || v.any_host(OL, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID, H2TAP_OL_AMOUNT}))
+                     ? launch_q18_probe_tma : launch_q18_probe)(colp<int32_t>(v, OL, H2TAP_OL_W_ID), colp<int32_t>(v, OL, H2TAP_OL_D_ID),
+                                 colp<int32_t>(v, OL, H2TAP_OL_O_ID), colp<int64_t>(v, OL, H2TAP_OL_AMOUNT),
+                                 n_ol, s, e->num_sms, e->compute);
+        });
+    }
     CK(cudaGetLastError());
     q.zone = q18_zone(v, false);
     q.view = &v;
@@ -1982,6 +2014,17 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
             ctx[i6].shared_scan = 1;
             ctx[i6].shared_cutoff = ctx[i1].p[0];
             ctx[i1].shared_scan = 2;
+            // the full pass: one Q18 after them, and no Q3 (it shares Q18's
+            // scratch, which the pass fills ahead of Q18's own launch) — Q18's probe joins the pass
+            int i18 = -1, n18 = 0, n3 = 0;
+            for (uint32_t i = 0; i < n; ++i) {
+                if (ctx[i].plan == H2TAP_Q18) { i18 = (int)i; ++n18; }
+                if (ctx[i].plan == H2TAP_Q3) ++n3;
+            }
+            if (e->full_pass && n18 == 1 && n3 == 0 && i18 > i1 && v->col[OL][H2TAP_OL_W_ID] &&
+                v->col[OL][H2TAP_OL_D_ID] && v->col[OL][H2TAP_OL_O_ID] &&
+                scan_tma_ok(e, *v, {H2TAP_OL_W_ID, H2TAP_OL_D_ID, H2TAP_OL_O_ID}))
+                ctx[i6].full18 = &ctx[i18];
         }
     }
     bool profile = false;
@@ -2051,7 +2094,9 @@ h2tap_status queries_impl(h2tap_engine *e, const h2tap_query *qs, uint32_t n, h2
         QueryCtx &q = ctx[i];
         for (size_t j = done; j < i; ++j)
             if (scratch_group(ctx[j].plan) == scratch_group(q.plan)) { finish_upto(i); break; }
-        q.r.reset(new_result(e, *v, q.flags & H2TAP_RESULT_DEVICE));
+        if (!q.r) q.r.reset(new_result(e, *v, q.flags & H2TAP_RESULT_DEVICE));
+        if (q.full18 && !q.full18->r)  // the full pass plans Q18's join indexes (plan_flags)
+            q.full18->r.reset(new_result(e, *v, q.full18->flags & H2TAP_RESULT_DEVICE));
         q.small = e->host_pool->get(256);
         CK(cudaHostGetDevicePointer(&q.small_dev, q.small.first, 0));
         if (!q.begin) {
@@ -2191,6 +2236,7 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
         if (const char *z = std::getenv("H2TAP_ZC_TMA")) e->zc_tma = std::atoi(z) != 0;
         if (const char *hu = std::getenv("H2TAP_HAVING_UNROLL")) e->having_unroll = std::atoi(hu) == 4 ? 4 : 2;
         if (const char *ss = std::getenv("H2TAP_SHARED_SCAN")) e->shared_scan = std::atoi(ss) != 0;
+        if (const char *fp = std::getenv("H2TAP_FULL_PASS")) e->full_pass = std::atoi(fp) != 0;
         if (const char *impl = std::getenv("H2TAP_PROBE")) e->probe_tma = std::strcmp(impl, "tma") == 0;
         if (const char *impl = std::getenv("H2TAP_COW")) e->cow_full = std::strcmp(impl, "full") == 0;
 

@@ -54,11 +54,14 @@ __device__ __forceinline__ bool jx_identity(const JoinIndex &j) {
     return j.dense && j.may_ident && __ldg(j.viol) == 0u;
 }
 
-__device__ __forceinline__ unsigned int jx_lookup(const JoinIndex &j, int w, int d, int id) {
+// `ident` = jx_identity(j), read once per kernel by callers in a hot loop (the verdict is a global
+// load: one L1 round trip per lookup otherwise, and an L2 one when a kernel's shared memory leaves
+// L1 little room)
+__device__ __forceinline__ unsigned int jx_lookup(const JoinIndex &j, int w, int d, int id, bool ident) {
     if (j.dense) {
         unsigned long long s;
         if (!dense_slot(j, w, d, id, s)) return kNoRow;  // outside the build box: no match
-        if (jx_identity(j)) return (unsigned int)s;       // clustered build side: positional
+        if (ident) return (unsigned int)s;                // clustered build side: positional
         return __ldcg(j.slots + s);
     }
     unsigned long long key;
@@ -70,6 +73,10 @@ __device__ __forceinline__ unsigned int jx_lookup(const JoinIndex &j, int w, int
         if (s.x == kEmpty) return kNoRow;
         h = (h + 1) & j.mask;
     }
+}
+
+__device__ __forceinline__ unsigned int jx_lookup(const JoinIndex &j, int w, int d, int id) {
+    return jx_lookup(j, w, d, id, jx_identity(j));
 }
 
 __host__ __device__ __forceinline__ uint64_t jx_words(const JoinIndex &j) {  // 16-byte units

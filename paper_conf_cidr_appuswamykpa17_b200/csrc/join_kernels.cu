@@ -163,6 +163,7 @@ q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ o
                  Q18Scratch s) {
     pdl_wait();
     pdl_trigger();
+    const bool ident = jx_identity(s.jo);  // after the wait: the verify kernel wrote the verdict
     const int lane = threadIdx.x & 31;
     const uint64_t gwarp = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
@@ -196,12 +197,12 @@ q18_probe_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict__ o
         } else {
             for (int j = 0; j < 4; ++j) { k[j] = {0, 0, 0}; a[j] = 0; }
         }
-        probe_lane_group<kFilter>(s, k, a, valid, lane);
+        probe_lane_group<kFilter>(s, k, a, valid, lane, ident);
     }
     // ragged tail (< 4 rows) plus nothing else: one thread, row at a time
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         for (uint64_t i = nvec * 4; i < n; ++i)
-            flush_run<kFilter>(s, Key3{ol_w[i], ol_d[i], ol_o[i]}, ol_amt[i], 1u);
+            flush_run<kFilter>(s, Key3{ol_w[i], ol_d[i], ol_o[i]}, ol_amt[i], 1u, ident);
     }
 }
 
@@ -224,6 +225,7 @@ q18_probe_tma_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict
     extern __shared__ __align__(128) unsigned char smem_raw[];
     ProbeStages &P = *reinterpret_cast<ProbeStages *>(smem_raw);
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const bool ident = jx_identity(s.jo);
     if (threadIdx.x == 0) {
         for (int st = 0; st < kProbeStages; ++st) {
             mbar_init(&P.full[st], 1);
@@ -277,10 +279,10 @@ q18_probe_tma_kernel(const int32_t *__restrict__ ol_w, const int32_t *__restrict
         // rows of a partial last group (< 4, last chunk only) go one by one, straight from smem
         if (!valid && r < rows)
             for (unsigned j = r; j < rows; ++j)
-                flush_run<false>(s, Key3{P.w[st][j], P.d[st][j], P.o[st][j]}, P.amt[st][j], 1u);
+                flush_run<false>(s, Key3{P.w[st][j], P.d[st][j], P.o[st][j]}, P.amt[st][j], 1u, ident);
         __syncwarp();
         if (lane == 0) mbar_arrive(&P.empty[st]);  // registers hold everything from here on
-        probe_lane_group<false>(s, k, a, valid, lane);
+        probe_lane_group<false>(s, k, a, valid, lane, ident);
     }
 }
 

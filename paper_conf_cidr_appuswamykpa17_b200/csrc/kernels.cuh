@@ -34,12 +34,14 @@ void launch_q6_tma(const int64_t *deliv, const int32_t *qty, const int64_t *amt,
 // warp-aggregated shared-memory atomics into a per-block hash table, then a global hash table.
 constexpr int kQ1Dense = 16;
 constexpr int kQ1GlobalSlots = 1 << 16;  // max distinct groups per rank
+constexpr unsigned kQ1GlobalUsed = 2u;    // Q1Scratch::flags: a group entered the global table
+constexpr unsigned kQ1Emitted = 4u;       // Q1Scratch::flags: the compact wrote the output
 struct Q1Group { long long key; long long cnt, qty, amt; };  // 32 B, compacted group
 struct Q1Scratch {
     unsigned long long *dense;   // [kQ1Dense * 3]: cnt, qty, amt per dense key
     unsigned long long *gtag;    // [kQ1GlobalSlots]: 0 = empty, else (1<<32 | (u32)key)
     unsigned long long *gacc;    // [kQ1GlobalSlots * 3]
-    unsigned int *flags;         // [1]: bit0 = global table full
+    unsigned int *flags;         // [1]: bit0 = global table full, kQ1GlobalUsed, kQ1Emitted
     Q1Group *groups;             // [kQ1GlobalSlots + kQ1Dense] compacted groups
     unsigned long long *ngroups; // [1]
     // output (ranked by key)
@@ -180,6 +182,12 @@ void launch_q18_probe(const int32_t *ol_w, const int32_t *ol_d, const int32_t *o
 void launch_q18_probe_tma(const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o,
                           const int64_t *ol_amt, uint64_t n_ol, const Q18Scratch &s, int num_sms,
                           cudaStream_t st);  // same result, TMA-bulk staged, one block per SM
+// the batch's full pass: Q6 + Q1 (as launch_q61_tma) and Q18's probe + group-join (K4) over one
+// TMA-staged read of order_line's 7 columns; the orders join index must be built
+void launch_q6118_tma(const int32_t *number, const int64_t *deliv, const int32_t *qty, const int64_t *amt,
+                      const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o, uint64_t n, int64_t cutoff,
+                      const Q1Scratch &s, int64_t d_lo, int64_t d_hi, int64_t q_lo, int64_t q_hi,
+                      const Q6Scratch &s6, const Q18Scratch &s18, int num_sms, cudaStream_t st);
 void launch_q18_having(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id,
                        const int32_t *o_c, const int32_t *o_cnt, const int64_t *o_ent,
                        uint64_t n_o, const int32_t *c_last, int64_t having,

@@ -31,19 +31,21 @@ __device__ __forceinline__ unsigned int keep_row(const Q18Scratch &s, unsigned i
 
 template <bool kFilter>
 __device__ __forceinline__ void flush_run(const Q18Scratch &s, const Key3 &k, long long sum,
-                                          unsigned int cnt) {
-    const unsigned int row = keep_row<kFilter>(s, jx_lookup(s.jo, k.w, k.d, k.o));
+                                          unsigned int cnt, bool ident) {
+    const unsigned int row = keep_row<kFilter>(s, jx_lookup(s.jo, k.w, k.d, k.o, ident));
     if (row != kNoRow) {
         atomicAdd(reinterpret_cast<unsigned long long *>(&s.acc[row].sum), (unsigned long long)sum);
         atomicAdd(&s.acc[row].cnt, cnt);
     }
 }
 
-// One warp step over 128 consecutive rows, 4 per lane (k, a in registers; `valid` per lane):
+// One warp step over 128 consecutive rows, 4 per lane (k, a in registers; `valid` per lane;
+// `ident` = jx_identity(s.jo), read once by the caller):
 // in-lane runs, cross-lane segmented scan, one probe + two atomics per run (see above).
 template <bool kFilter>
 __device__ __forceinline__ void probe_lane_group(const Q18Scratch &s, const Key3 (&k)[4],
-                                                 const long long (&a)[4], bool valid, int lane) {
+                                                 const long long (&a)[4], bool valid, int lane,
+                                                 bool ident) {
         // in-lane runs: b[j] = row j starts a run; s[j], c[j] = running sum / count of its run
         bool b1 = !eq3(k[1], k[0]), b2 = !eq3(k[2], k[1]), b3 = !eq3(k[3], k[2]);
         long long s0 = a[0], s1 = (b1 ? 0 : s0) + a[1], s2 = (b2 ? 0 : s1) + a[2], s3 = (b3 ? 0 : s2) + a[3];
@@ -89,7 +91,7 @@ __device__ __forceinline__ void probe_lane_group(const Q18Scratch &s, const Key3
             const Key3 kj = j == 0 ? k[0] : j == 1 ? k[1] : j == 2 ? k[2] : k[3];
             const long long sj = j == 0 ? fs[0] : j == 1 ? fs[1] : j == 2 ? fs[2] : fs[3];
             const unsigned cj = j == 0 ? fc[0] : j == 1 ? fc[1] : j == 2 ? fc[2] : fc[3];
-            const unsigned int row = keep_row<kFilter>(s, jx_lookup(s.jo, kj.w, kj.d, kj.o));
+            const unsigned int row = keep_row<kFilter>(s, jx_lookup(s.jo, kj.w, kj.d, kj.o, ident));
             if (row != kNoRow) {
                 atomicAdd(reinterpret_cast<unsigned long long *>(&s.acc[row].sum), (unsigned long long)sj);
                 atomicAdd(&s.acc[row].cnt, cj);

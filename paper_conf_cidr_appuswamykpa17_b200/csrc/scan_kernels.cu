@@ -15,6 +15,7 @@
 #include "bulk_pipeline.cuh"
 #include "kernels.cuh"
 #include "peer.cuh"
+#include "probe_device.cuh"
 
 namespace h2tap {
 namespace {
@@ -282,6 +283,7 @@ __device__ void q1_global_add(const Q1Scratch &g, unsigned long long tag, unsign
     for (int p = 0; p < kQ1GlobalSlots; ++p) {
         const unsigned long long prev = atomicCAS(g.gtag + h, 0ull, tag);
         if (prev == 0ull || prev == tag) {
+            if (prev == 0ull) atomicOr(g.flags, kQ1GlobalUsed);  // the compact must scan the table
             atomicAdd(g.gacc + 3 * h + 0, c);
             atomicAdd(g.gacc + 3 * h + 1, (unsigned long long)q);
             atomicAdd(g.gacc + 3 * h + 2, (unsigned long long)a);
@@ -465,44 +467,95 @@ q1_kernel(const int4 *__restrict__ number, const longlong2 *__restrict__ deliv,
 // (120 KB): thread-private dense slots, warp-aggregated sparse path (as q1_kernel). 12 warps
 // instead of 8: the slot updates are latency-bound.
 constexpr int kQ1Chunk = 1024;
-template <int kS> struct Q1StagesT {
-    long long deliv[kS][kQ1Chunk];
-    long long amt[kS][kQ1Chunk];
-    int number[kS][kQ1Chunk];
-    int qty[kS][kQ1Chunk];
+// the full pass's extra columns (Q18's join keys), present only in the probe variant
+template <int kS, int kC, bool kP> struct ScanKeysT {};
+template <int kS, int kC> struct ScanKeysT<kS, kC, true> { int w[kS][kC], d[kS][kC], o[kS][kC]; };
+template <int kS, int kC = kQ1Chunk, bool kP = false> struct Q1StagesT {
+    long long deliv[kS][kC];
+    long long amt[kS][kC];
+    int number[kS][kC];
+    int qty[kS][kC];
+    ScanKeysT<kS, kC, kP> key;
     uint64_t full[kS], empty[kS];
 };
-// Q1 alone: 8 aggregating warps, 5 stages (208 KB). Shared with Q6: 12 aggregating warps (their
+// Q1 alone: 12 aggregating warps, 4 stages (216 KB). Shared with Q6: 12 aggregating warps (their
 // latency-bound slot updates were the shared pass's limit) and 4 stages (224 KB).
-template <bool kQ6> struct Q1TmaCfg {
-    static constexpr int kW = 12;                             // aggregating warps
+constexpr int kQ6SideWarps = 6;
+// The full pass's geometry (build-time constants for A/B variants,
+// scripts/build_variants.py). Measured at W = 100 (pass time): 12 Q1 warps / 3 stages / 7 probe
+// warps 297 us — each probe warp must finish one ~300-instruction step per chunk, a latency chain
+// of shuffles; two probe groups taking alternate chunks 200-206 us; 8 Q1 warps / 4 stages / 896-row
+// chunks / 2 x 7 probe warps / 4 Q6 warps 191 us (the default); 768-row chunks x 5 stages 208 us,
+// 6 Q1 warps x 5 stages 211 us; a try_wait suspend hint: no change.
+#ifndef H2TAP_FULL_DIAG
+#define H2TAP_FULL_DIAG 0   // A/B diagnosis only: 1 = the probe warps skip their step (wrong Q18)
+#endif
+#ifndef H2TAP_FULL_W
+#define H2TAP_FULL_W 8      // Q1 aggregating warps
+#endif
+#ifndef H2TAP_FULL_S
+#define H2TAP_FULL_S 4      // ring stages
+#endif
+#ifndef H2TAP_FULL_C
+#define H2TAP_FULL_C 896    // rows per chunk (a multiple of 128: one probe warp step per 128 rows)
+#endif
+#ifndef H2TAP_FULL_PG
+#define H2TAP_FULL_PG 2     // probe warp groups; group g takes the chunks it == g (mod PG)
+#endif
+#ifndef H2TAP_FULL_Q6W
+#define H2TAP_FULL_Q6W 4    // Q6 side warps in the full pass
+#endif
+#ifndef H2TAP_FULL_SLEEP_NS
+#define H2TAP_FULL_SLEEP_NS 0  // consumer waits: try_wait suspend-time hint (0: none)
+#endif
+template <bool kQ6, bool kProbe = false> struct Q1TmaCfg {
+    static constexpr int kW = kProbe ? H2TAP_FULL_W : 12;           // aggregating warps
     static constexpr int kT = kW * 32;
-    static constexpr int kS = 4;                              // ring stages
+    static constexpr int kS = kProbe ? H2TAP_FULL_S : 4;            // ring stages
+    static constexpr int kC = kProbe ? H2TAP_FULL_C : kQ1Chunk;     // rows per chunk
+    static constexpr int kQ6W = kQ6 ? (kProbe ? H2TAP_FULL_Q6W : kQ6SideWarps) : 0;  // Q6 side warps
+    static constexpr int kPG = kProbe ? H2TAP_FULL_PG : 1;            // probe warp groups
+    static constexpr int kPW = kProbe ? kC / 128 : 0;                // Q18 probe warps per group
+    static constexpr int kThreads = (kW + 1 + kQ6W + kPG * kPW) * 32;
+    using Stages = Q1StagesT<kS, kC, kProbe>;
+    static constexpr size_t kSmem = sizeof(Stages) + sizeof(Q1SmemT<kT>);
+    static_assert(!kProbe || kC % 128 == 0, "probe warps take 128-row steps");
 };
 
 // kQ6: shared scan of a batch's Q6 and Q1 — Q6 reads a subset of Q1's columns
 // (ol_delivery_d, ol_quantity, ol_amount), so the same staged chunk also feeds Q6's predicate and
 // sum; the block tail adds Q6's reduction (as q6_tma_kernel). One pass over 24 B/row instead of
 // 20 + 24.
-// Shared-scan block: warps 0-7 Q1 (as above), warp 8 the producer, warps 9-12 Q6 on the same
+// Shared-scan block: warps 0-11 Q1, warp 12 the producer, then the Q6 side warps on the same
 // staged chunks (registers only) — Q6 added to the Q1 warps' rows lengthened their dependent
 // shared-memory update chains (145 vs 117 us); separate warps run it alongside.
-constexpr int kQ6SideWarps = 6;
-constexpr int kQ61Threads = (Q1TmaCfg<true>::kW + 1 + kQ6SideWarps) * 32;
-template <bool kQ6>
-__global__ void __launch_bounds__(kQ6 ? kQ61Threads : (Q1TmaCfg<false>::kW + 1) * 32, 1)
+// kProbe (the batch's full pass): the chunks also carry Q18's join keys
+// (ol_w_id, ol_d_id, ol_o_id) and kC / 128 probe warps run the K4 warp step (probe_device.cuh)
+// on them: the batch reads order_line once, 36 B/row, instead of 24 + 20 B/row (ol_amount is
+// shared by all three queries). The orders join index must be built before the pass.
+constexpr int kQ61Threads = Q1TmaCfg<true>::kThreads;
+template <bool kQ6, bool kProbe = false>
+__global__ void __launch_bounds__(Q1TmaCfg<kQ6, kProbe>::kThreads, 1)
 q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deliv,
               const int *__restrict__ qty, const long long *__restrict__ amt, uint64_t n,
               long long cutoff, Q1Scratch g, Q6Pred pred6, long long *__restrict__ part6,
               unsigned int *__restrict__ counter6, long long *__restrict__ out6,
-              long long *__restrict__ host_out6) {
+              long long *__restrict__ host_out6, const int *__restrict__ ol_w,
+              const int *__restrict__ ol_d, const int *__restrict__ ol_o, Q18Scratch ps) {
     pdl_wait();
     pdl_trigger();
     extern __shared__ __align__(128) unsigned char smem_raw[];
-    using Cfg = Q1TmaCfg<kQ6>;
-    constexpr int kQ1W = Cfg::kW, kQ1T = Cfg::kT, kQ1Stages = Cfg::kS;
-    Q1StagesT<kQ1Stages> &P = *reinterpret_cast<Q1StagesT<kQ1Stages> *>(smem_raw);
-    Q1SmemT<kQ1T> &sm = *reinterpret_cast<Q1SmemT<kQ1T> *>(smem_raw + sizeof(Q1StagesT<kQ1Stages>));
+    using Cfg = Q1TmaCfg<kQ6, kProbe>;
+    constexpr int kQ1W = Cfg::kW, kQ1T = Cfg::kT, kQ1Stages = Cfg::kS, kC = Cfg::kC;
+    constexpr int kQ6W = Cfg::kQ6W, kPW = Cfg::kPW, kPG = Cfg::kPG;
+    typename Cfg::Stages &P = *reinterpret_cast<typename Cfg::Stages *>(smem_raw);
+    Q1SmemT<kQ1T> &sm = *reinterpret_cast<Q1SmemT<kQ1T> *>(smem_raw + sizeof(typename Cfg::Stages));
+    auto wait_full = [&](int s, int it) {
+        if constexpr (kProbe && H2TAP_FULL_SLEEP_NS > 0)
+            mbar_wait_hint(&P.full[s], (unsigned)(it / kQ1Stages) & 1u, H2TAP_FULL_SLEEP_NS);
+        else
+            mbar_wait(&P.full[s], (unsigned)(it / kQ1Stages) & 1u);
+    };
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     long long sum6 = 0, cnt6 = 0;  // kQ6 only
     if (tid < kQ1T) {
@@ -515,13 +568,13 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
     if (tid == 0) {
         for (int s = 0; s < kQ1Stages; ++s) {
             mbar_init(&P.full[s], 1);
-            mbar_init(&P.empty[s], kQ1W + (kQ6 ? kQ6SideWarps : 0));
+            mbar_init(&P.empty[s], kQ1W + kQ6W + kPW);
         }
         fence_mbar_init();
         if (blockIdx.x == 0) *g.ngroups = 0;  // consumed by q1_compact (stream-ordered)
     }
     __syncthreads();
-    const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
+    const uint64_t nchunks = (n + kC - 1) / kC;
     if (warp == kQ1W) {  // producer
         if (lane == 0) {
             const uint64_t pol = policy_evict_first();
@@ -530,17 +583,62 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
                 const int s = it % kQ1Stages;
                 const unsigned ph = (unsigned)(it / kQ1Stages) & 1u;
                 if (it >= kQ1Stages) mbar_wait(&P.empty[s], ph ^ 1u);
-                const uint64_t r0 = c * kQ1Chunk;
-                const unsigned rows = (unsigned)(n - r0 < (uint64_t)kQ1Chunk ? n - r0 : (uint64_t)kQ1Chunk);
+                const uint64_t r0 = c * kC;
+                const unsigned rows = (unsigned)(n - r0 < (uint64_t)kC ? n - r0 : (uint64_t)kC);
                 const unsigned b8 = round16(rows * 8), b4 = round16(rows * 4);
-                mbar_arrive_expect_tx(&P.full[s], 2 * b8 + 2 * b4);
+                mbar_arrive_expect_tx(&P.full[s], 2 * b8 + (kProbe ? 5 : 2) * b4);
                 bulk_g2s(P.deliv[s], deliv + r0, b8, &P.full[s], pol);
                 bulk_g2s(P.amt[s], amt + r0, b8, &P.full[s], pol);
                 bulk_g2s(P.number[s], number + r0, b4, &P.full[s], pol);
                 bulk_g2s(P.qty[s], qty + r0, b4, &P.full[s], pol);
+                if constexpr (kProbe) {
+                    bulk_g2s(P.key.w[s], ol_w + r0, b4, &P.full[s], pol);
+                    bulk_g2s(P.key.d[s], ol_d + r0, b4, &P.full[s], pol);
+                    bulk_g2s(P.key.o[s], ol_o + r0, b4, &P.full[s], pol);
+                }
             }
         }
-    } else if (kQ6 && warp > kQ1W) {  // Q6 side warps: 128 threads, 4 row pairs each
+    } else if (kProbe && warp > kQ1W + kQ6W) {  // Q18 probe warps: one 128-row step per chunk each
+      if constexpr (kProbe) {
+        using namespace pd;
+        const bool ident = jx::jx_identity(ps.jo);  // read once (after pdl_wait: verify has run)
+        const int pw = (warp - (kQ1W + 1 + kQ6W)) % kPW, pg = (warp - (kQ1W + 1 + kQ6W)) / kPW;
+        static_assert(kPW == kC / 128, "one 128-row step per probe warp per chunk");
+        int it = pg;
+        for (uint64_t c = blockIdx.x + (uint64_t)pg * gridDim.x; c < nchunks; c += (uint64_t)kPG * gridDim.x, it += kPG) {
+            const int s = it % kQ1Stages;
+            wait_full(s, it);
+            const unsigned rows = (unsigned)(n - c * kC < (uint64_t)kC ? n - c * kC : (uint64_t)kC);
+            const unsigned r = pw * 128 + lane * 4;  // this lane's 4 consecutive rows
+            Key3 k[4];
+            long long a[4];
+            const bool valid = r + 3 < rows;
+            if (valid) {
+                const int4 W = *reinterpret_cast<const int4 *>(&P.key.w[s][r]);
+                const int4 D = *reinterpret_cast<const int4 *>(&P.key.d[s][r]);
+                const int4 O = *reinterpret_cast<const int4 *>(&P.key.o[s][r]);
+                const longlong2 A0 = *reinterpret_cast<const longlong2 *>(&P.amt[s][r]);
+                const longlong2 A1 = *reinterpret_cast<const longlong2 *>(&P.amt[s][r + 2]);
+                k[0] = {W.x, D.x, O.x}; k[1] = {W.y, D.y, O.y}; k[2] = {W.z, D.z, O.z}; k[3] = {W.w, D.w, O.w};
+                a[0] = A0.x; a[1] = A0.y; a[2] = A1.x; a[3] = A1.y;
+            } else {
+                for (int j = 0; j < 4; ++j) { k[j] = {0, 0, 0}; a[j] = 0; }
+            }
+            // rows of a partial last group (< 4, last chunk only) go one by one
+            if (!valid && r < rows)
+                for (unsigned j = r; j < rows; ++j)
+                    flush_run<false>(ps, Key3{P.key.w[s][j], P.key.d[s][j], P.key.o[s][j]}, P.amt[s][j], 1u, ident);
+            // the stage is released before the step (the step works on registers)
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&P.empty[s]);
+#if H2TAP_FULL_DIAG != 1
+            probe_lane_group<false>(ps, k, a, valid, lane, ident);
+#else
+            if (a[0] == 0x7fffffffffffffffll && k[0].w == 12345) probe_lane_group<false>(ps, k, a, valid, lane, ident);
+#endif
+        }
+      }
+    } else if (kQ6 && warp > kQ1W) {  // Q6 side warps: 4 row pairs each
         // the predicate as two unsigned range tests (same result as Q6Pred: a NULL date is
         // INT64_MIN, below every lower bound > INT64_MIN; an empty range passes nothing)
         const long long dlo = pred6.d_lo > kNullTs ? pred6.d_lo : kNullTs + 1;
@@ -556,12 +654,10 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
         int it = 0;
         for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
             const int s = it % kQ1Stages;
-            mbar_wait(&P.full[s], (unsigned)(it / kQ1Stages) & 1u);
-            const unsigned rows = (unsigned)(n - c * kQ1Chunk < (uint64_t)kQ1Chunk ? n - c * kQ1Chunk
-                                                                                 : (uint64_t)kQ1Chunk);
-            if (rows == (unsigned)kQ1Chunk) {  // full chunk: 128-bit / 64-bit shared loads of pairs
-                constexpr int kPairs = kQ1Chunk / 2, kStep = kQ6SideWarps * 32;
-                static_assert(kPairs % kStep == 0 || kQ6SideWarps != 4, "full-chunk pair loop");
+            wait_full(s, it);
+            const unsigned rows = (unsigned)(n - c * kC < (uint64_t)kC ? n - c * kC : (uint64_t)kC);
+            if (rows == (unsigned)kC) {  // full chunk: 128-bit / 64-bit shared loads of pairs
+                constexpr int kPairs = kC / 2, kStep = kQ6W * 32;
 #pragma unroll
                 for (int k = 0; k < (kPairs + kStep - 1) / kStep; ++k) {
                     const unsigned pr = t6 + k * kStep;
@@ -574,7 +670,7 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
                     c32 += (unsigned)p0 + (unsigned)p1;
                 }
             } else {
-                for (unsigned r = t6; r < rows; r += kQ6SideWarps * 32) {
+                for (unsigned r = t6; r < rows; r += kQ6W * 32) {
                     const bool p0 = pass(P.deliv[s][r], P.qty[s][r]);
                     sum6 += p0 ? P.amt[s][r] : 0;
                     c32 += p0;
@@ -588,12 +684,11 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
         int it = 0;
         for (uint64_t c = blockIdx.x; c < nchunks; c += gridDim.x, ++it) {
             const int s = it % kQ1Stages;
-            mbar_wait(&P.full[s], (unsigned)(it / kQ1Stages) & 1u);
-            const unsigned rows = (unsigned)(n - c * kQ1Chunk < (uint64_t)kQ1Chunk ? n - c * kQ1Chunk
-                                                                                 : (uint64_t)kQ1Chunk);
+            wait_full(s, it);
+            const unsigned rows = (unsigned)(n - c * kC < (uint64_t)kC ? n - c * kC : (uint64_t)kC);
             // all four rows' loads first: the stage and the tables share one shared-memory
             // buffer, so loads after a table store would wait for it (possible aliasing)
-            constexpr int kU = (kQ1Chunk + kQ1T - 1) / kQ1T;
+            constexpr int kU = (kC + kQ1T - 1) / kQ1T;
             int keys[kU], qs[kU];
             long long ds[kU], as[kU];
 #pragma unroll
@@ -630,7 +725,7 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
     __syncthreads();
     q1_block_merge<kQ1T>(sm, g, tid);
     if (kQ6) {  // Q6: block reduction -> per-block partial -> last block folds (q6_tma_kernel)
-        constexpr int kW = kQ61Threads / 32;
+        constexpr int kW = Cfg::kThreads / 32;
         __shared__ long long s_sum[kW], s_cnt[kW];
         __shared__ bool s_last;
         sum6 = warp_sum(sum6);
@@ -665,11 +760,38 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
     }
 }
 
-// Collect the dense and global tables into groups[] and clear them for the next query.
+// Collect the dense and global tables into groups[] and clear them for the next query. When no
+// group reached the global table (kQ1GlobalUsed clear: every key was dense, the TPC-C case) block
+// 0 alone does it and also writes the ranked output (dense keys are already in key order), and
+// q1_emit only publishes the counts (kQ1Emitted): one warp instead of a 64 K-slot scan + rank.
 __global__ void q1_compact_kernel(Q1Scratch g) {
     pdl_wait();
     pdl_trigger();
+    if (!(*reinterpret_cast<volatile unsigned int *>(g.flags) & kQ1GlobalUsed)) {
+        if (blockIdx.x != 0 || threadIdx.x >= 32) return;
+        const int lane = threadIdx.x;
+        unsigned long long c = 0, qs = 0, as = 0;
+        if (lane < kQ1Dense) { c = g.dense[3 * lane]; qs = g.dense[3 * lane + 1]; as = g.dense[3 * lane + 2]; }
+        const unsigned present = __ballot_sync(kFull, c != 0);
+        if (c) {
+            const int r = __popc(present & ((1u << lane) - 1u));  // rank = key order
+            g.groups[r] = Q1Group{(long long)lane, (long long)c, (long long)qs, (long long)as};
+            g.o_key[r] = lane;
+            g.o_qty[r] = (long long)qs;
+            g.o_amt[r] = (long long)as;
+            g.o_cnt[r] = (long long)c;
+            g.o_avg_qty[r] = (double)(long long)qs / (double)(long long)c;
+            g.o_avg_amt[r] = ((double)(long long)as / (double)(long long)c) / 100.0;
+            g.dense[3 * lane] = g.dense[3 * lane + 1] = g.dense[3 * lane + 2] = 0;
+        }
+        if (lane == 0) {
+            *g.ngroups = __popc(present);
+            atomicOr(g.flags, kQ1Emitted);
+        }
+        return;
+    }
     const uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    if (i == 0) atomicAnd(g.flags, ~kQ1Emitted);
     if (i < (uint64_t)kQ1Dense) {
         const unsigned long long c = g.dense[3 * i];
         if (c) {
@@ -691,9 +813,6 @@ __global__ void q1_compact_kernel(Q1Scratch g) {
     }
 }
 
-// Multi-GPU (a7): every rank pushed its compacted group list into this rank's
-// mailbox (launch_peer_push) and launch_peer_wait saw all of them arrive; fold every list (this
-// rank's included) into the clean global table; q1_compact + q1_emit then run as on one GPU.
 __global__ void __launch_bounds__(256) q1_peer_merge_kernel(PeerArgs p, Q1Scratch g) {
     pdl_wait();
     pdl_trigger();
@@ -722,10 +841,15 @@ __global__ void q1_emit_kernel(Q1Scratch g) {
     pdl_trigger();
     __shared__ long long tile[1024];
     const uint64_t ng = *g.ngroups;  // read on the device: no host round trip before emitting
-    if (g.host_small && blockIdx.x == 0 && threadIdx.x == 0) {  // mapped pinned: no D2H copies
-        g.host_small[0] = ng;
-        reinterpret_cast<unsigned int *>(g.host_small)[2] = *g.flags;
+    const unsigned fl = *reinterpret_cast<volatile unsigned int *>(g.flags);
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
+        if (g.host_small) {  // mapped pinned: no D2H copies
+            g.host_small[0] = ng;
+            reinterpret_cast<unsigned int *>(g.host_small)[2] = fl & 1u;
+        }
+        atomicAnd(g.flags, ~kQ1GlobalUsed);  // the compact has emptied the global table
     }
+    if (fl & kQ1Emitted) return;  // the compact wrote the output (dense keys only)
     if ((uint64_t)blockIdx.x * blockDim.x >= ng) return;  // grid sized for the maximum
     const uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
     const long long mine = i < ng ? g.groups[i].key : 0;
@@ -813,12 +937,11 @@ void launch_q1_tma(const int32_t *number, const int64_t *deliv, const int32_t *q
                    const int64_t *amt, uint64_t n, int64_t cutoff, const Q1Scratch &s, int num_sms,
                    cudaStream_t st) {
     using Cfg = Q1TmaCfg<false>;
-    const size_t smem = sizeof(Q1StagesT<Cfg::kS>) + sizeof(Q1SmemT<Cfg::kT>);
-    const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
+    const uint64_t nchunks = (n + Cfg::kC - 1) / Cfg::kC;
     const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)scan_sms(num_sms)));
-    launch_pdl(q1_tma_kernel<false>, grid, (Q1TmaCfg<false>::kW + 1) * 32, smem, st, number, reinterpret_cast<const long long *>(deliv), qty,
+    launch_pdl(q1_tma_kernel<false>, grid, Cfg::kThreads, Cfg::kSmem, st, number, reinterpret_cast<const long long *>(deliv), qty,
                reinterpret_cast<const long long *>(amt), n, cutoff, s, Q6Pred{0, 0, 0, 0}, nullptr, nullptr,
-               nullptr, nullptr);
+               nullptr, nullptr, nullptr, nullptr, nullptr, Q18Scratch{});
     count_launches(1);
 }
 
@@ -827,12 +950,25 @@ void launch_q61_tma(const int32_t *number, const int64_t *deliv, const int32_t *
                     int64_t d_hi, int64_t q_lo, int64_t q_hi, const Q6Scratch &s6, int num_sms,
                     cudaStream_t st) {
     using Cfg = Q1TmaCfg<true>;
-    const size_t smem = sizeof(Q1StagesT<Cfg::kS>) + sizeof(Q1SmemT<Cfg::kT>);
-    const uint64_t nchunks = (n + kQ1Chunk - 1) / kQ1Chunk;
+    const uint64_t nchunks = (n + Cfg::kC - 1) / Cfg::kC;
     const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)scan_sms(num_sms)));
-    launch_pdl(q1_tma_kernel<true>, grid, kQ61Threads, smem, st, number, reinterpret_cast<const long long *>(deliv),
+    launch_pdl(q1_tma_kernel<true>, grid, Cfg::kThreads, Cfg::kSmem, st, number, reinterpret_cast<const long long *>(deliv),
                qty, reinterpret_cast<const long long *>(amt), n, cutoff, s, Q6Pred{d_lo, d_hi, q_lo, q_hi},
-               s6.block_part, s6.done_counter, s6.out, s6.host_out);
+               s6.block_part, s6.done_counter, s6.out, s6.host_out, nullptr, nullptr, nullptr, Q18Scratch{});
+    count_launches(1);
+}
+
+void launch_q6118_tma(const int32_t *number, const int64_t *deliv, const int32_t *qty, const int64_t *amt,
+                      const int32_t *ol_w, const int32_t *ol_d, const int32_t *ol_o, uint64_t n, int64_t cutoff,
+                      const Q1Scratch &s, int64_t d_lo, int64_t d_hi, int64_t q_lo, int64_t q_hi,
+                      const Q6Scratch &s6, const Q18Scratch &s18, int num_sms, cudaStream_t st) {
+    using Cfg = Q1TmaCfg<true, true>;
+    const uint64_t nchunks = (n + Cfg::kC - 1) / Cfg::kC;
+    const unsigned grid = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(nchunks, (uint64_t)scan_sms(num_sms)));
+    launch_pdl(q1_tma_kernel<true, true>, grid, Cfg::kThreads, Cfg::kSmem, st, number,
+               reinterpret_cast<const long long *>(deliv), qty, reinterpret_cast<const long long *>(amt), n, cutoff,
+               s, Q6Pred{d_lo, d_hi, q_lo, q_hi}, s6.block_part, s6.done_counter, s6.out, s6.host_out, ol_w, ol_d,
+               ol_o, s18);
     count_launches(1);
 }
 
@@ -871,6 +1007,7 @@ cudaError_t set_attributes_scan(int num_sms) {
         (const void *)q1_peer_merge_kernel,
         (const void *)q1_tma_kernel<false>,
         (const void *)q1_tma_kernel<true>,
+        (const void *)q1_tma_kernel<true, true>,
         (const void *)q6_kernel,
         (const void *)q6_tma_kernel};
     const cudaError_t le = force_load(kKernels, sizeof kKernels / sizeof kKernels[0]);
@@ -883,10 +1020,13 @@ cudaError_t set_attributes_scan(int num_sms) {
         e = cudaFuncSetAttribute(q1_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(Q1Smem));
     if (e == cudaSuccess)
         e = cudaFuncSetAttribute(q1_tma_kernel<false>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                 (int)(sizeof(Q1StagesT<Q1TmaCfg<false>::kS>) + sizeof(Q1SmemT<Q1TmaCfg<false>::kT>)));
+                                 (int)Q1TmaCfg<false>::kSmem);
     if (e == cudaSuccess)
         e = cudaFuncSetAttribute(q1_tma_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                 (int)(sizeof(Q1StagesT<Q1TmaCfg<true>::kS>) + sizeof(Q1SmemT<Q1TmaCfg<true>::kT>)));
+                                 (int)Q1TmaCfg<true>::kSmem);
+    if (e == cudaSuccess)
+        e = cudaFuncSetAttribute(q1_tma_kernel<true, true>, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                 (int)Q1TmaCfg<true, true>::kSmem);
     return e;
 }
 

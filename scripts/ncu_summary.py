@@ -75,6 +75,7 @@ if traffic:
              "bucket_local_emit_kernel<8192, 2048, 1>": "q18_bucket_sort_emit_large",
              "q18_plan_kernel": "q18_plan", "q1_compact_kernel": "q1_compact",
              "q1_emit_kernel": "q1_emit", "q1_tma_kernel<1>": "q61_shared_scan",
+             "q1_tma_kernel<1, 0>": "q61_shared_scan", "q1_tma_kernel<1, 1>": "q6118_full_pass",
              "q18_acc_stats_kernel": "q18_acc_stats", "q18_having_rec_kernel": "q18_having_records",
              "ob_scatter_rec_kernel": "q18_bucket_scatter",
              "bucket_local_emit_kernel<1536, 0, 1>": "q18_bucket_sort_emit",

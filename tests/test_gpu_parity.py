@@ -800,3 +800,47 @@ def test_q18_clustered_index_verification(L, layout, order_mode):
     got3 = L.q(3, [Q3_LO, 0x4100])
     for k in want3:
         assert np.array_equal(got3[k], want3[k]), k
+
+
+@pytest.mark.parametrize("layout", ["clustered", "shuffled"])
+@pytest.mark.parametrize("full", ["1", "0"])
+def test_full_pass_batch(h, monkeypatch, order_mode, layout, full):
+    """The batch's full pass: a Q6, Q1, Q18 batch reads order_line once — the
+    shared Q6 + Q1 scan also stages Q18's keys and runs its probe. Ragged sizes around the 896-row
+    chunk and the 4-row lane group, random parameters (HAVING exactly at a group's sum too),
+    positional (clustered) and slot-array (shuffled orders) join indexes, the hash-join plan and
+    both ORDER BY layouts, vs the oracle; H2TAP_FULL_PASS=0 runs the probe as its own kernel."""
+    monkeypatch.setenv("H2TAP_FULL_PASS", full)
+    e = h.h2tap_open(0)
+    try:
+        rng = np.random.default_rng(91)
+        base = chgen.generate(1, 3, seed=91)
+        if layout == "shuffled":
+            perm = rng.permutation(len(base["orders"]["o_id"]))
+            base["orders"] = {k: v[perm].copy() for k, v in base["orders"].items()}
+        epoch = 0
+        for n_keep in (100_003, 897, 896, 895, 130, 5, 1):
+            t = dict(base)
+            t["order_line"] = {k: v[:n_keep].copy() for k, v in base["order_line"].items()}
+            epoch += 1
+            h.h2tap_load_snapshot(e, h.hot_path_tables(t), epoch)
+            sums = oracle.q18(t, -(2**62))["amount_sum"]
+            thrs = [Q18_HAVING, int(sums[len(sums) // 2]) if len(sums) else 0]
+            for k, thr in enumerate(thrs):
+                d_lo = int(rng.integers(chgen.TS_1995, chgen.TS_2025))
+                p6 = [d_lo, int(rng.integers(d_lo, chgen.TS_2025 + 10**12)), int(rng.integers(0, 6)),
+                      int(rng.integers(4, 12))]
+                cut = int(rng.integers(chgen.TS_1995, chgen.TS_2025))
+                f18 = HASH if k == 1 else 0
+                rs = h.h2tap_run_queries(e, [(6, p6, 0), (1, [cut], 0), (18, [thr], f18)])
+                got = []
+                for r in rs:
+                    x = r.to_numpy()
+                    x["_nulls"] = dict(r.nulls)
+                    got.append(x)
+                    h.h2tap_free(r)
+                assert_q6(got[0], oracle.q6(t, *p6))
+                assert_q1(got[1], oracle.q1(t, cut))
+                assert_q18(got[2], oracle.q18(t, thr))
+    finally:
+        h.h2tap_close(e)
