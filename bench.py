@@ -906,7 +906,8 @@ def main():
                               if flush is not None else "inputs > L2 (no flush)")},
             "latency_ms": dict({f"{q}_in_batch": round(v, 4) for q, v in lat_max.items()},
                                q6_alone=round(q6_alone_ms, 4), q1_alone=round(q1_alone_ms, 4),
-                               **({"q6_q1_shared_scan_batch": round(lat_max["q6"] + lat_max["q1"], 4)}
+                               **({("q6_q1_q18probe_full_pass_batch" if full_pass else "q6_q1_shared_scan_batch"):
+                                   round(lat_max["q6"] + lat_max["q1"], 4)}
                                   if "q6" in lat_max and "q1" in lat_max else {})),
             "step_ms_median": round(step_p50, 5), "step_ms_p99": round(step_p99, 5),
             "c2": ({"workload": "CH Q1 alone at W=100 per GPU (BASELINE configs[1]), device time (query's own events), "

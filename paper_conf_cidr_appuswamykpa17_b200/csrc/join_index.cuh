@@ -61,6 +61,7 @@ __device__ __forceinline__ unsigned int jx_lookup(const JoinIndex &j, int w, int
     if (j.dense) {
         unsigned long long s;
         if (!dense_slot(j, w, d, id, s)) return kNoRow;  // outside the build box: no match
+        H2TAP_CHECK(s < j.range);
         if (ident) return (unsigned int)s;                // clustered build side: positional
         return __ldcg(j.slots + s);
     }

@@ -391,6 +391,14 @@ void count_launches(int n);
 // (launch latency and its block scheduling overlap k's tail). Every such kernel starts with
 // pdl_wait() — it returns once the preceding grid has completed and its writes are visible — and
 // pdl_trigger(), which lets the next grid launch. H2TAP_PDL=0 launches them normally (A/B).
+// Device-side invariant checks, compiled in only for the checking build (-DH2TAP_CHECKS=1,
+// scripts/build_variants.py): a violated index bound traps the kernel (the test then fails with
+// a CUDA error) — the bounds checks that stand in for compute-sanitizer where it is unavailable.
+#if defined(H2TAP_CHECKS) && H2TAP_CHECKS
+#define H2TAP_CHECK(cond) do { if (!(cond)) __trap(); } while (0)
+#else
+#define H2TAP_CHECK(cond) do { } while (0)
+#endif
 __device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
 __device__ __forceinline__ void pdl_trigger() { asm volatile("griddepcontrol.launch_dependents;" ::: "memory"); }
 bool pdl_enabled();

@@ -610,6 +610,7 @@ q1_tma_kernel(const int *__restrict__ number, const long long *__restrict__ deli
             wait_full(s, it);
             const unsigned rows = (unsigned)(n - c * kC < (uint64_t)kC ? n - c * kC : (uint64_t)kC);
             const unsigned r = pw * 128 + lane * 4;  // this lane's 4 consecutive rows
+            H2TAP_CHECK(rows <= (unsigned)kC && (c * kC + rows <= n) && s < kQ1Stages);
             Key3 k[4];
             long long a[4];
             const bool valid = r + 3 < rows;

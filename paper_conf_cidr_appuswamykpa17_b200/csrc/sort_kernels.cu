@@ -714,6 +714,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
         for (unsigned int i = threadIdx.x; i < m; i += kT) {
             const unsigned long long kk = S.rec[i].x;
             const unsigned int p = atomicAdd(&S.cur[(unsigned int)(kk >> ssh) & smask], 1u);
+            H2TAP_CHECK(p < m);
             S.idx[p] = (unsigned short)i;
         }
         __syncthreads();
@@ -729,6 +730,7 @@ __device__ __forceinline__ void carry_sort_emit(const ulonglong2 *__restrict__ k
                     rank += (o.x < r.x) | ((o.x == r.x) & ((o.y < r.y) | ((o.y == r.y) & (j < i))));
                 }
             }
+            H2TAP_CHECK(rank < m && me < m);
             S.srt[rank] = (unsigned short)me;
         }
         __syncthreads();
@@ -1581,7 +1583,9 @@ ob_scatter_rec_kernel(const ulonglong2 *__restrict__ rec, uint64_t n_o, const Q1
         for (int u = 0; u < U; ++u) {
             const unsigned int i = i0 + u * kObThreads;
             if (i >= m) break;
+            H2TAP_CHECK((r[u].x >> shift) < (unsigned long long)nb && m <= r1 - r0);
             const unsigned int p = atomicAdd(&cur[(unsigned int)(r[u].x >> shift)], 1u);
+            H2TAP_CHECK(p < n_o);
             kv[p] = r[u];
         }
     }
