@@ -844,3 +844,30 @@ def test_full_pass_batch(h, monkeypatch, order_mode, layout, full):
                 assert_q18(got[2], oracle.q18(t, thr))
     finally:
         h.h2tap_close(e)
+
+
+@pytest.mark.parametrize("keys", ["dense", "one_sparse", "negative"])
+def test_q1_keys_in_shared_pass_batches(h, keys):
+    """Q1 inside the batch's shared / full pass with every ol_number dense, one key
+    just outside the dense range (16) and one negative key (the global-table path and the
+    general compact + emit), vs the oracle, in the bench's Q6 + Q1 + Q18 batch and in a Q6 + Q1
+    batch, repeated (the tables are cleared between queries)."""
+    t = chgen.generate(1, 3, seed=73)
+    ol = t["order_line"]
+    if keys == "one_sparse":
+        ol["ol_number"][12345] = 16
+    elif keys == "negative":
+        ol["ol_number"][777] = -3
+    e = h.h2tap_open(0)
+    try:
+        h.h2tap_load_snapshot(e, h.hot_path_tables(t), 1)
+        for batch in ([(6, None, 0), (1, None, 0), (18, None, 0)], [(6, None, 0), (1, [chgen.TS_1995], 0)],
+                      [(6, None, 0), (1, None, 0), (18, None, 0)]):
+            rs = h.h2tap_run_queries(e, batch)
+            g1 = rs[1].to_numpy()
+            for r in rs:
+                h.h2tap_free(r)
+            cut = batch[1][1][0] if batch[1][1] else Q1_CUTOFF
+            assert_q1(g1, oracle.q1(t, cut))
+    finally:
+        h.h2tap_close(e)
