@@ -1091,13 +1091,15 @@ ob_scan_kernel(unsigned int *__restrict__ mat, int G, int nb, unsigned int *__re
                ulonglong2 *__restrict__ touch = nullptr, uint64_t touch_n = 0) {
     pdl_wait();
     pdl_trigger();
+    const unsigned nscan = (unsigned)(nb + 31) / 32;  // the column-scan blocks (launch nb)
     if (plan && plan->dist) nb = 1 << plan->bucket_bits;  // (grid sized for the launch nb)
-    if (touch) {  // v3: the scatter's target lines into L2 first (l2_touch_kernel; the scan has spare
-                  // bandwidth: it is latency-bound)
+    if (blockIdx.x >= nscan) {  // v3: blocks past the scan write the scatter's target lines into
+        // L2 (evict_last) while the latency-bound scan runs on the first nscan blocks
         const uint64_t keep = l2_policy_evict_last();
-        const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-        for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < touch_n; i += stride)
+        const uint64_t stride = (uint64_t)(gridDim.x - nscan) * blockDim.x;
+        for (uint64_t i = (uint64_t)(blockIdx.x - nscan) * blockDim.x + threadIdx.x; i < touch_n; i += stride)
             st16_policy(touch + i, 0ull, 0ull, keep);
+        return;
     }
     extern __shared__ unsigned int tile[];  // [G][32]; the last block reuses it for nb totals
     __shared__ bool last;
@@ -1129,7 +1131,7 @@ ob_scan_kernel(unsigned int *__restrict__ mat, int G, int nb, unsigned int *__re
     }
     __threadfence();
     __syncthreads();
-    if (threadIdx.x == 0) last = atomicAdd(ticket, 1u) == gridDim.x - 1;
+    if (threadIdx.x == 0) last = atomicAdd(ticket, 1u) == nscan - 1;
     __syncthreads();
     if (!last) return;
     __threadfence();
@@ -1621,8 +1623,8 @@ void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, c
     count_launches(1);
     end();
     begin("q18_sort_scan");
-    launch_pdl(ob_scan_kernel, (nb + 31) / 32, 32 * kScanWarps, 4 * std::max(32 * G, nb), st, bs.mat, G, nb,
-               bs.count, bs.offset, bs.ticket, plan,
+    launch_pdl(ob_scan_kernel, (nb + 31) / 32 + (kv_touch_mode() == 1 ? num_sms : 0), 32 * kScanWarps,
+               4 * std::max(32 * G, nb), st, bs.mat, G, nb, bs.count, bs.offset, bs.ticket, plan,
                kv_touch_mode() == 1 ? reinterpret_cast<ulonglong2 *>(bs.kv) : nullptr, kv_touch_mode() == 1 ? n_o : 0);
     count_launches(1);
     end();
@@ -1908,9 +1910,9 @@ void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long lo
     }
     begin("q18_sort_scan");
     const bool tin = hv && kv_touch_mode() == 1;
-    launch_pdl(ob_scan_kernel, (nb + 31) / 32, 32 * kScanWarps, 4 * std::max(32 * G, nb), st, s.mat, G, nb, s.count,
-               s.offset, s.ticket, (const Q18Plan *)plan, tin ? reinterpret_cast<ulonglong2 *>(s.kv) : nullptr,
-               tin ? hv->n_o : (uint64_t)0);
+    launch_pdl(ob_scan_kernel, (nb + 31) / 32 + (tin ? num_sms : 0), 32 * kScanWarps, 4 * std::max(32 * G, nb), st,
+               s.mat, G, nb, s.count, s.offset, s.ticket, (const Q18Plan *)plan,
+               tin ? reinterpret_cast<ulonglong2 *>(s.kv) : nullptr, tin ? hv->n_o : (uint64_t)0);
     count_launches(1);
     end();
     begin("q18_dist_counts");
