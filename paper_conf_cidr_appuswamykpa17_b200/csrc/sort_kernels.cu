@@ -1490,6 +1490,7 @@ q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict
     const int shift = s_shift;
     const Q18SortSpec sp = S;
     const uint64_t keep = l2_policy_evict_last();  // records are re-read by the scatter
+    const bool ident_c = jx::jx_identity(s.jc);     // read once (the verify kernel ran before)
     constexpr int U = 4;
     if (s_carry)
     for (uint64_t base = r0; base < r1; base += (uint64_t)U * kHrThreads) {
@@ -1513,7 +1514,7 @@ q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict
         }
 #pragma unroll
         for (int u = 0; u < U; ++u)  // customer ⋈ orders, independent across rows
-            if (crow[u] == 0u) crow[u] = jx::jx_lookup(s.jc, w[u], d[u], c[u]);
+            if (crow[u] == 0u) crow[u] = jx::jx_lookup(s.jc, w[u], d[u], c[u], ident_c);
         ulonglong2 rc[U];
 #pragma unroll
         for (int u = 0; u < U; ++u) {
