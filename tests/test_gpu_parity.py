@@ -819,7 +819,7 @@ def test_full_pass_batch(h, monkeypatch, order_mode, layout, full):
             perm = rng.permutation(len(base["orders"]["o_id"]))
             base["orders"] = {k: v[perm].copy() for k, v in base["orders"].items()}
         epoch = 0
-        for n_keep in (100_003, 897, 896, 895, 130, 5, 1):
+        for n_keep in (100_003, 897, 896, 895, 130, 5, 1, 0):
             t = dict(base)
             t["order_line"] = {k: v[:n_keep].copy() for k, v in base["order_line"].items()}
             epoch += 1
@@ -869,5 +869,31 @@ def test_q1_keys_in_shared_pass_batches(h, keys):
                 h.h2tap_free(r)
             cut = batch[1][1][0] if batch[1][1] else Q1_CUTOFF
             assert_q1(g1, oracle.q1(t, cut))
+    finally:
+        h.h2tap_close(e)
+
+
+@pytest.mark.parametrize("empty", ["all", "order_line", "orders", "customer"])
+def test_full_pass_batch_empty_tables(h, empty):
+    """The full-pass batch (Q6 + Q1 + Q18 in one order_line read) over empty
+    tables: every table, or one of order_line / orders / customer emptied (the others full) —
+    vs the oracle (NULL revenue, no Q1 groups, no Q18 rows where nothing joins)."""
+    t = chgen.generate(1, 1 if empty == "all" else 2, seed=19)
+    if empty != "all":
+        t[empty] = {k: v[:0].copy() for k, v in t[empty].items()}
+    e = h.h2tap_open(0)
+    try:
+        h.h2tap_load_snapshot(e, h.hot_path_tables(t), 1)
+        for _ in range(2):
+            rs = h.h2tap_run_queries(e, [(6, None, 0), (1, None, 0), (18, [-100], 0)])
+            got = []
+            for r in rs:
+                x = r.to_numpy()
+                x["_nulls"] = dict(r.nulls)
+                got.append(x)
+                h.h2tap_free(r)
+            assert_q6(got[0], oracle.q6(t, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI))
+            assert_q1(got[1], oracle.q1(t, Q1_CUTOFF))
+            assert_q18(got[2], oracle.q18(t, -100))
     finally:
         h.h2tap_close(e)
