@@ -1644,7 +1644,8 @@ void finish_q18(h2tap_engine *e, QueryCtx &q) {
     const char *const *names = q3 ? kQ3Names : kQ18Names;
     const uint32_t *types = q3 ? kQ3Types : kQ18Types;
     const int ncols = q3 ? 5 : 8;
-    if (q.v3 && !q.dist && (sm->tie & (1u | 2u | 4u | 8u))) q18_rerun_v2(e, q);  // (carry did not fit)
+    // (carry did not fit, a bucket overflowed, or the direct ORDER BY counted a row with no customer)
+    if (q.v3 && !q.dist && (sm->tie & (1u | 2u | 4u | 8u | 16u))) q18_rerun_v2(e, q);
     const unsigned int err = sm->err;  // world > 1: every rank's join errors and the exchange's
     const unsigned pl = q.plan;
     if (err & kPeerErrTimeout) {

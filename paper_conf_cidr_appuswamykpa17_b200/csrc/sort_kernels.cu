@@ -616,6 +616,8 @@ constexpr int kLcCapLarge = 8192;  // carry records per bucket in the large inst
 // so the only global traffic is the bucket's records in and the result columns out. The next
 // bucket's first kPre * 256 records are loaded into registers while the current one is
 // decoded and stored, and its sub-bucket counters are cleared then too (one barrier less).
+constexpr unsigned int kFlagHoles = 16u;    // direct ORDER BY: a counted row found no customer (the
+                                            // host re-runs the v2 path; the emits skip their work)
 constexpr int kPre = 3;
 // kT threads per block, at most kSub sub-buckets per bucket (a power of two).
 template <int kCap, int kMin, int kSub = kLsSubMax, int kT = kEmThreads>
@@ -789,6 +791,7 @@ bucket_local_emit_kernel(const unsigned long long *__restrict__ k, const unsigne
                          unsigned int *big, int sub_log2 = 3, PeerArgs pa = PeerArgs{}) {
     pdl_wait();
     pdl_trigger();
+    if (flag && (*reinterpret_cast<volatile unsigned int *>(flag) & kFlagHoles)) return;  // re-run on v2
     extern __shared__ __align__(16) unsigned char smem_raw[];
     if (pa.world > 1) {  // distributed ORDER BY: this rank's buckets, exchanged into its heap
         // (their arrival was awaited by the one-thread peer_wait launched before this grid)
@@ -983,6 +986,7 @@ carry_large_emit_kernel(const unsigned long long *__restrict__ k, const unsigned
                         int sub_log2, PeerArgs pa) {
     pdl_wait();
     pdl_trigger();
+    if (flag && (*reinterpret_cast<volatile unsigned int *>(flag) & kFlagHoles)) return;  // re-run on v2
     extern __shared__ __align__(16) unsigned char smem_raw[];
     if (pa.world > 1) {  // distributed ORDER BY: this rank's buckets in its heap (as the emit above)
         const unsigned long long xs = plan->xseq;
@@ -1459,13 +1463,15 @@ q18_acc_stats_kernel(const Q18Acc *__restrict__ acc, const int64_t *__restrict__
 // range (the same partition the scatter uses): records are compacted into the block's own range
 // of rec[] (a shared counter per warp-ballot), the block's bucket counts become matrix row p.
 constexpr int kHrThreads = 512;  // 2 blocks per SM (<= 64 registers), 4 rows per thread in flight
+template <bool kDirect>
 __global__ void __launch_bounds__(kHrThreads, 2)
 q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict__ o_d,
                       const int32_t *__restrict__ o_id, const int32_t *__restrict__ o_c,
                       const int32_t *__restrict__ o_cnt, const int64_t *__restrict__ o_ent, uint64_t n_o,
                       const int32_t *__restrict__ c_last, long long having, Q18Scratch s,
                       const Q18Plan *__restrict__ plan, int nb_launch, unsigned int *__restrict__ mat,
-                      unsigned int *__restrict__ cnt_part, ulonglong2 *__restrict__ rec, unsigned int *flag) {
+                      unsigned int *__restrict__ cnt_part, ulonglong2 *__restrict__ rec, unsigned int *flag,
+                      const unsigned int *__restrict__ offset) {
     pdl_wait();
     pdl_trigger();
     extern __shared__ unsigned int h[];
@@ -1482,10 +1488,15 @@ q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict
     }
     __syncthreads();
     const int nb = s_nb;
-    for (int i = threadIdx.x; i < nb; i += kHrThreads) h[i] = 0;
-    __syncthreads();
     uint64_t r0, r1;
     ob_range(n_o, r0, r1);
+    if (kDirect) {  // h[] = this partition's cursors: bucket start + the lower partitions' counts
+        const unsigned int *mrow = mat + (uint64_t)blockIdx.x * nb;
+        for (int i = threadIdx.x; i < nb; i += kHrThreads) h[i] = offset[i] + mrow[i];
+    } else {
+        for (int i = threadIdx.x; i < nb; i += kHrThreads) h[i] = 0;
+    }
+    __syncthreads();
     const int lane = threadIdx.x & 31;
     const int shift = s_shift;
     const Q18SortSpec sp = S;
@@ -1497,6 +1508,7 @@ q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict
         long long sum[U], ent[U];
         int w[U], d[U], c[U], oid[U], cnt[U];
         unsigned int crow[U];
+        bool hv_pass[U];
 #pragma unroll
         for (int u = 0; u < U; ++u) {  // independent coalesced loads first
             const uint64_t r = base + (uint64_t)u * kHrThreads + threadIdx.x;
@@ -1513,8 +1525,10 @@ q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict
             }
         }
 #pragma unroll
-        for (int u = 0; u < U; ++u)  // customer ⋈ orders, independent across rows
+        for (int u = 0; u < U; ++u) {  // customer ⋈ orders, independent across rows
+            hv_pass[u] = crow[u] == 0u;
             if (crow[u] == 0u) crow[u] = jx::jx_lookup(s.jc, w[u], d[u], c[u], ident_c);
+        }
         ulonglong2 rc[U];
 #pragma unroll
         for (int u = 0; u < U; ++u) {
@@ -1528,8 +1542,23 @@ q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict
             row.o_w_id = w[u];
             row.o_d_id = d[u];
             rc[u] = carry_record(row, sum[u], sp);
-            atomicAdd(&h[(unsigned int)(rc[u].x >> shift)], 1u);
+            if (kDirect) {  // straight to its final bucket position (the scatter's job)
+                const unsigned int p = atomicAdd(&h[(unsigned int)(rc[u].x >> shift)], 1u);
+                H2TAP_CHECK(p < n_o);
+                st16_policy(rec + p, rc[u].x, rc[u].y, keep);
+            } else {
+                atomicAdd(&h[(unsigned int)(rc[u].x >> shift)], 1u);
+            }
         }
+        if (kDirect) {
+#pragma unroll
+            for (int u = 0; u < U; ++u) {
+                // counted by q18_acc_hist (cnt > 0, sum > having) but no customer: a hole
+                if (crow[u] == kNoRow && hv_pass[u]) atomicOr(flag, kFlagHoles);
+                const unsigned int bal = __ballot_sync(kFull, crow[u] != kNoRow);
+                if (bal && lane == __ffs(bal) - 1) atomicAdd(&s_cnt, (unsigned int)__popc(bal));
+            }
+        } else
 #pragma unroll
         for (int u = 0; u < U; ++u) {  // warp-aggregated compaction into the block's range
             const bool v = crow[u] != kNoRow;
@@ -1542,12 +1571,77 @@ q18_having_rec_kernel(const int32_t *__restrict__ o_w, const int32_t *__restrict
         }
     }
     __syncthreads();
-    unsigned int *row = mat + (uint64_t)blockIdx.x * nb;
-    for (int i = threadIdx.x; i < nb; i += kHrThreads) row[i] = h[i];
+    if (!kDirect) {
+        unsigned int *row = mat + (uint64_t)blockIdx.x * nb;
+        for (int i = threadIdx.x; i < nb; i += kHrThreads) row[i] = h[i];
+    }
     if (threadIdx.x == 0) {
-        cnt_part[blockIdx.x] = s_cnt;
+        if (!kDirect) cnt_part[blockIdx.x] = s_cnt;
         if (s_cnt) atomicAdd(s.nout, (unsigned long long)s_cnt);
     }
+}
+
+// The direct ORDER BY's count pass (one GPU): per row partition (the HAVING pass's),
+// the bucket counts of the groups passing HAVING (cnt > 0, sum > having; the customer join is
+// assumed — a missing customer is a hole the HAVING pass reports), so that HAVING writes each
+// record at its final bucket position and no scatter pass is needed. When the bucket bits lie
+// inside field a (the usual plan) only acc[] is read.
+__global__ void __launch_bounds__(kObThreads)
+q18_acc_hist_kernel(const Q18Acc *__restrict__ acc, const int32_t *__restrict__ o_w,
+                    const int32_t *__restrict__ o_d, const int32_t *__restrict__ o_id,
+                    const int64_t *__restrict__ o_ent, uint64_t n_o, long long having,
+                    const Q18Plan *__restrict__ plan, int nb, unsigned int *__restrict__ mat,
+                    unsigned int *big) {
+    pdl_wait();
+    pdl_trigger();
+    extern __shared__ unsigned int h[];
+    if (big && blockIdx.x == 0 && threadIdx.x == 0) *big = 0;  // the emit's oversized-bucket list
+    for (int i = threadIdx.x; i < nb; i += kObThreads) h[i] = 0;
+    __syncthreads();
+    const Q18SortSpec sp = plan->spec;
+    const int shift = plan->shift;
+    const bool amt_only = shift >= sp.prefix_bits - sp.bits_a;
+    uint64_t r0, r1;
+    ob_range(n_o, r0, r1);
+    if (sp.carry && amt_only) {  // acc[] only, 8 independent loads in flight per thread
+        constexpr int U = 8;
+        const int sa = shift - (sp.prefix_bits - sp.bits_a);
+        for (uint64_t r = r0 + threadIdx.x; r < r1; r += (uint64_t)U * kObThreads) {
+            ulonglong2 a[U];
+#pragma unroll
+            for (int u = 0; u < U; ++u) {
+                const uint64_t x = r + (uint64_t)u * kObThreads;
+                a[u] = x < r1 ? __ldcs(reinterpret_cast<const ulonglong2 *>(acc + x)) : make_ulonglong2(0, 0);
+            }
+#pragma unroll
+            for (int u = 0; u < U; ++u) {
+                const long long sum = (long long)a[u].x;
+                if ((unsigned int)a[u].y > 0 && sum > having) {
+                    const unsigned int b = (unsigned int)(field_a(sum, sp) >> sa);
+                    H2TAP_CHECK(b < (unsigned int)nb);
+                    atomicAdd(&h[b], 1u);
+                }
+            }
+        }
+    } else if (sp.carry)
+    for (uint64_t r = r0 + threadIdx.x; r < r1; r += kObThreads) {
+        const ulonglong2 a = __ldcs(reinterpret_cast<const ulonglong2 *>(acc + r));
+        const long long sum = (long long)a.x;
+        if (!((unsigned int)a.y > 0 && sum > having)) continue;
+        unsigned int b;
+        {
+            Q18Row row{};
+            row.o_entry_d = __ldg(o_ent + r);
+            row.o_w_id = __ldg(o_w + r); row.o_d_id = __ldg(o_d + r); row.o_id = __ldg(o_id + r);
+            row.c_last = sp.cl_min; row.c_id = sp.ci_min; row.o_ol_cnt = sp.n_min;
+            b = (unsigned int)(carry_record(row, sum, sp).x >> shift);
+        }
+        H2TAP_CHECK(b < (unsigned int)nb);
+        atomicAdd(&h[b], 1u);
+    }
+    __syncthreads();
+    unsigned int *row = mat + (uint64_t)blockIdx.x * nb;
+    for (int i = threadIdx.x; i < nb; i += kObThreads) row[i] = h[i];
 }
 
 // Each block's records (rec[r0 .. r0 + cnt_part[p])) to their bucket positions: the shared cursors
@@ -1618,9 +1712,33 @@ void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, c
     auto end = [&] { if (marks) marks->end(); };
     const int nb = 1 << bucket_bits;
     const int G = ob_grid(num_sms);
+    // direct (default, H2TAP_ORDER_DIRECT=0 for the scatter pass): counts from acc[] first, the
+    // column scan, then HAVING writes every record at its final bucket position
+    const char *dx = std::getenv("H2TAP_ORDER_DIRECT");  // (read per query: tests switch it)
+    const bool direct = !(dx && dx[0] == '0');
+    if (direct) {
+        begin("q18_bucket_count");
+        launch_pdl(q18_acc_hist_kernel, G, kObThreads, 4 * nb, st, (const Q18Acc *)s.acc, o_w, o_d, o_id, o_ent, n_o,
+                   (long long)having, plan, nb, bs.mat, bs.big);
+        count_launches(1);
+        end();
+        begin("q18_sort_scan");
+        launch_pdl(ob_scan_kernel, (nb + 31) / 32 + (kv_touch_mode() == 1 ? num_sms : 0), 32 * kScanWarps,
+                   4 * std::max(32 * G, nb), st, bs.mat, G, nb, bs.count, bs.offset, bs.ticket, plan,
+                   kv_touch_mode() == 1 ? reinterpret_cast<ulonglong2 *>(bs.kv) : nullptr, kv_touch_mode() == 1 ? n_o : 0);
+        count_launches(1);
+        end();
+        begin("q18_having_records");
+        launch_pdl(q18_having_rec_kernel<true>, G, kHrThreads, 4 * nb, st, o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o,
+                   c_last, (long long)having, s, plan, nb, bs.mat, cnt_part, reinterpret_cast<ulonglong2 *>(bs.kv),
+                   flag, (const unsigned int *)bs.offset);
+        count_launches(1);
+        end();
+    } else {
     begin("q18_having_records");
-    launch_pdl(q18_having_rec_kernel, G, kHrThreads, 4 * nb, st, o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o, c_last,
-               (long long)having, s, plan, nb, bs.mat, cnt_part, reinterpret_cast<ulonglong2 *>(bs.k[0]), flag);
+    launch_pdl(q18_having_rec_kernel<false>, G, kHrThreads, 4 * nb, st, o_w, o_d, o_id, o_c, o_cnt, o_ent, n_o, c_last,
+               (long long)having, s, plan, nb, bs.mat, cnt_part, reinterpret_cast<ulonglong2 *>(bs.k[0]), flag,
+               (const unsigned int *)nullptr);
     count_launches(1);
     end();
     begin("q18_sort_scan");
@@ -1641,7 +1759,8 @@ void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, c
                reinterpret_cast<ulonglong2 *>(bs.kv), bs.big);
     count_launches(1);
     end();
-    // (big[], the oversized-bucket work list, was reset by the scatter kernel)
+    }
+    // (big[], the oversized-bucket work list, was reset by the count or the scatter kernel)
     static const int sub_log2 = [] {
         const char *v = std::getenv("H2TAP_SUB_ROWS_LOG2");
         return v ? std::max(0, std::min(6, std::atoi(v))) : 1;
@@ -1898,9 +2017,10 @@ void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long lo
     end();
     if (hv) {  // v3: HAVING builds the carry records and the bucket counts with the global plan
         begin("q18_having_records");
-        launch_pdl(q18_having_rec_kernel, G, kHrThreads, nb * 4, st, hv->o_w, hv->o_d, hv->o_id, hv->o_c, hv->o_cnt,
+        launch_pdl(q18_having_rec_kernel<false>, G, kHrThreads, nb * 4, st, hv->o_w, hv->o_d, hv->o_id, hv->o_c, hv->o_cnt,
                    hv->o_ent, hv->n_o, hv->c_last, (long long)hv->having, hv->s, (const Q18Plan *)plan, nb, s.mat,
-                   hv->cnt_part, reinterpret_cast<ulonglong2 *>(s.k[0]), flag);
+                   hv->cnt_part, reinterpret_cast<ulonglong2 *>(s.k[0]), flag,
+                   (const unsigned int *)nullptr);
         count_launches(1);
         end();
     } else {
@@ -2014,7 +2134,9 @@ cudaError_t set_attributes_sort(int num_sms) {
         (const void *)q18_plan_kernel,
         (const void *)scatter_kernel,
         (const void *)q18_acc_stats_kernel,
-        (const void *)q18_having_rec_kernel,
+        (const void *)q18_having_rec_kernel<false>,
+        (const void *)q18_having_rec_kernel<true>,
+        (const void *)q18_acc_hist_kernel,
         (const void *)ob_scatter_rec_kernel,
         (const void *)l2_touch_kernel,
         (const void *)carry_large_emit_kernel};
@@ -2033,7 +2155,9 @@ cudaError_t set_attributes_sort(int num_sms) {
         {(const void *)ob_scatter_kernel, 4 << kBucketMaxBits},
         {(const void *)ob_scan_kernel, 4 * std::max(32 * G, 1 << kBucketMaxBits)},
         {(const void *)q18_dist_route_kernel, 4 << kBucketMaxBits},
-        {(const void *)q18_having_rec_kernel, 4 << kBucketMaxBits},
+        {(const void *)q18_having_rec_kernel<false>, 4 << kBucketMaxBits},
+        {(const void *)q18_having_rec_kernel<true>, 4 << kBucketMaxBits},
+        {(const void *)q18_acc_hist_kernel, 4 << kBucketMaxBits},
         {(const void *)carry_large_emit_kernel, (int)kLgSmem},
         {(const void *)ob_scatter_rec_kernel, 4 << kBucketMaxBits},
     };

@@ -62,7 +62,7 @@ def L(h, eng):
     return Loader(h, eng)
 
 
-@pytest.fixture(params=["carry", "rowid"])
+@pytest.fixture(params=["carry", "rowid", "scatter"])
 def order_mode(request, monkeypatch):
     """The ORDER BY's two record layouts: 128-bit carry records (default when
     the row fits) and (64-bit prefix, row id) pairs with tie-fix / exact fallback."""
@@ -70,6 +70,10 @@ def order_mode(request, monkeypatch):
         monkeypatch.setenv("H2TAP_ORDER_CARRY", "0")
     else:
         monkeypatch.delenv("H2TAP_ORDER_CARRY", raising=False)
+    if request.param == "scatter":  # carry records through the staged HAVING output + scatter pass
+        monkeypatch.setenv("H2TAP_ORDER_DIRECT", "0")
+    else:
+        monkeypatch.delenv("H2TAP_ORDER_DIRECT", raising=False)
     return request.param
 
 
@@ -425,9 +429,11 @@ def test_profile_reports_kernels(h, eng, L):
     L.load(t)
     r = h.h2tap_run_query(eng, h.H2TAP_Q18, flags=h.H2TAP_QUERY_PROFILE)
     names = [k for k, _ in r.kernels]
-    # v3 ORDER BY: the HAVING pass writes the carry records
-    assert {"q18_build", "q18_probe_groupjoin", "q18_acc_stats", "q18_having_records", "q18_bucket_scatter",
-            "q18_bucket_sort_emit"} <= set(names)
+    # v3 ORDER BY: bucket counts from the accumulators, the column scan, then the
+    # HAVING pass writes each carry record at its final bucket position (no scatter pass)
+    assert {"q18_build", "q18_probe_groupjoin", "q18_acc_stats", "q18_bucket_count", "q18_sort_scan",
+            "q18_having_records", "q18_bucket_sort_emit"} <= set(names)
+    assert "q18_bucket_scatter" not in names
     assert all(ms >= 0 for _, ms in r.kernels) and r.device_ms > 0
     r.free()
 
