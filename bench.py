@@ -226,6 +226,7 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None, clustered=F
                 "q18_bucket_scatter": (16 + 16) * n_pass,
                 # direct ORDER BY (default): bucket counts from the accumulators alone
                 "q18_bucket_count": 16 * n_o,
+                "q18_plan_count": 16 * n_o,  # plan + counts in one kernel: acc[] once (L2 re-read)
                 "q18_bucket_sort_emit": (16 + 40) * n_pass}.get(kernel)
     if box:
         slots_o, slots_c, slot_b = box[0], box[1], 4
@@ -252,6 +253,7 @@ def alg_bytes(kernel, n_ol, n_o, n_c, n_pass, sort_passes, box=None, clustered=F
         # ORDER BY v2 (default): count matrix + scatter computing keys + chunked local sort
         "q18_sort_hist": 8 * n_pass,                       # amounts (bucket bits inside field a)
         "q18_bucket_count": 16 * n_o,                      # direct ORDER BY: counts from acc[]
+        "q18_plan_count": 16 * n_o,                        # plan + counts, one kernel
         "q18_bucket_scatter": (16 + 16) * n_pass if sort_passes == "carry"
                               else (40 + 16) * n_pass if sort_passes != "v1" else (12 + 12) * n_pass,
         # v3 (default): the accumulators for the plan's amount bounds (o_entry_d: zone map)

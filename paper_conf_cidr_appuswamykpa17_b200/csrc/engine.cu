@@ -30,6 +30,20 @@
 #include "../../include/h2tap.h"
 #include "kernels.cuh"
 
+// engines open per device in this process (a kernel with a grid barrier needs its grid alone on
+// the device: two such grids from two engines could each hold part of the SMs and wait forever)
+static std::mutex g_dev_mu;
+static std::map<int, int> g_dev_engines;
+static void engines_on_device_add(int dev, int d) {
+    std::lock_guard<std::mutex> g(g_dev_mu);
+    g_dev_engines[dev] += d;
+}
+static int engines_on_device(int dev) {
+    std::lock_guard<std::mutex> g(g_dev_mu);
+    auto it = g_dev_engines.find(dev);
+    return it == g_dev_engines.end() ? 0 : it->second;
+}
+
 namespace h2tap {
 static std::atomic<uint64_t> g_launches{0};
 void count_launches(int n) { g_launches.fetch_add((uint64_t)n, std::memory_order_relaxed); }
@@ -1456,6 +1470,18 @@ void q18_launch_v3(h2tap_engine *e, const View &v, QueryCtx &q) {
         bb = std::max(1, std::min(kBucketMaxBits, bb + std::atoi(d)));
     q18_alloc_out(e, q, n_max);
     const Q18PlanArgs pa{s.stats, q.zone, nullptr, 1};
+    // the plan and the bucket counts in one kernel (grid barrier): direct ORDER BY, o_entry_d's bounds
+    // from the zone map, the grid resident at once, no other engine on the device (§4.4)
+    const char *dx = std::getenv("H2TAP_ORDER_DIRECT"), *fx = std::getenv("H2TAP_PLAN_HIST");
+    const bool fused = !(dx && dx[0] == '0') && !(fx && fx[0] == '0') && q.zone.has_e &&
+                       engines_on_device(e->device) == 1 && q18_plan_hist_ok(e->num_sms, bb);
+    if (fused)
+        e->prof.run("q18_plan_count", [&] {
+            launch_q18_plan_hist(s, n_o, q.p[0], cpart,
+                                 static_cast<unsigned long long *>(e->arena.get("q18.gbar", 64, true, e->compute)),
+                                 scount, q.zone, bb, q.plan_dev, q.tie_dev, bs, e->num_sms, e->compute);
+        });
+    else
     e->prof.run("q18_acc_stats", [&] {
         launch_q18_acc_stats(s, o_ent, n_o, q.p[0], cpart, scount, &pa, bb, q.plan_dev, q.tie_dev, e->num_sms,
                              e->compute);
@@ -1463,7 +1489,7 @@ void q18_launch_v3(h2tap_engine *e, const View &v, QueryCtx &q) {
     q18_order_v3(colp<int32_t>(v, O, H2TAP_O_W_ID), colp<int32_t>(v, O, H2TAP_O_D_ID), colp<int32_t>(v, O, H2TAP_O_ID),
                  colp<int32_t>(v, O, H2TAP_O_C_ID), colp<int32_t>(v, O, H2TAP_O_OL_CNT), o_ent, n_o,
                  colp<int32_t>(v, C, H2TAP_C_LAST), q.p[0], s, q.plan_dev, bb, bs, cnt_part, q.out, q.tie_dev,
-                 e->num_sms, e->compute, &marks);
+                 e->num_sms, e->compute, &marks, fused);
     CK(cudaGetLastError());
     launch_q18_publish(s.nout, s.err, q.tie_dev, q.small_dev, s.jo, s.jc, e->compute);  // -> small (mapped)
 }
@@ -2304,6 +2330,7 @@ h2tap_status h2tap_open(const h2tap_config *cfg, h2tap_engine **out) {
             CK(cudaHostGetDevicePointer(&dp, P.err_host, 0));
             P.args.err_host = static_cast<unsigned int *>(dp);
         }
+        engines_on_device_add(e->device, 1);
         *out = e.release();
         return H2TAP_OK;
     });
@@ -2552,6 +2579,7 @@ void h2tap_free(h2tap_result *r) {
 
 void h2tap_close(h2tap_engine *e) {
     if (!e) return;
+    engines_on_device_add(e->device, -1);
     cudaSetDevice(e->device);
     try { publish_ready(e, true); } catch (...) {}
     cudaStreamSynchronize(e->compute);

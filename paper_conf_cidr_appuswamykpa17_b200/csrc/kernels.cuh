@@ -332,7 +332,15 @@ void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, c
                   const int32_t *o_cnt, const int64_t *o_ent, uint64_t n_o, const int32_t *c_last,
                   int64_t having, const Q18Scratch &s, const Q18Plan *plan, int bucket_bits,
                   const BucketSort &bs, unsigned int *cnt_part, const Q18Cols &dst, unsigned int *flag,
-                  int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr);
+                  int num_sms, cudaStream_t st, PhaseMarks *marks = nullptr, bool counted = false);
+// one GPU, direct ORDER BY: the plan (acc_stats) and the bucket counts in one kernel with a grid
+// barrier — only when its grid is resident at once (q18_plan_hist_ok) and no other engine shares
+// the device
+bool q18_plan_hist_ok(int num_sms, int bucket_bits);
+void launch_q18_plan_hist(const Q18Scratch &s, uint64_t n_o, int64_t having, unsigned long long *cpart,
+                          unsigned long long *gbar, unsigned long long *count, const Q18Zone &zone,
+                          int bucket_bits, Q18Plan *plan, unsigned int *flag, const BucketSort &bs, int num_sms,
+                          cudaStream_t st);
 // hv non-null: the v3 input (records built by the HAVING pass); null: rows + amounts (Q3)
 void q18_bucket_order_dist(const PeerArgs &pa, const Q18Row *rows, const long long *amt, Q18Plan *plan,
                            const Q18PlanArgs &meta, const unsigned int *err, const BucketSort &s,

@@ -1690,6 +1690,153 @@ ob_scatter_rec_kernel(const ulonglong2 *__restrict__ rec, uint64_t n_o, const Q1
 
 }  // namespace
 
+__device__ __forceinline__ unsigned long long ld_acquire_gpu_u64(const unsigned long long *a) {
+    unsigned long long v;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(a) : "memory");
+    return v;
+}
+
+// The plan and the bucket counts in one kernel (one GPU, direct ORDER BY): each
+// block reduces its row partition's passing amount bounds (as q18_acc_stats), a grid barrier (a
+// monotonic 64-bit arrival counter; the grid is one wave of resident blocks — the host checks the
+// occupancy and that no other engine shares the device), every block derives the same plan from
+// all blocks' partials (block 0 publishes it), then counts its partition's buckets (as
+// q18_acc_hist) re-reading acc[] while it is still in L2.
+constexpr int kPhThreads = 512;
+__global__ void __launch_bounds__(kPhThreads)
+q18_plan_hist_kernel(const Q18Acc *__restrict__ acc, uint64_t n_o, long long having, Q18Stats *part,
+                     unsigned long long *cpart, unsigned long long *gbar, Q18Stats *stats,
+                     unsigned long long *count, Q18Zone zone, int bucket_bits, Q18Plan *plan,
+                     unsigned int *flag, unsigned int *mat, unsigned int *big) {
+    pdl_wait();
+    pdl_trigger();
+    extern __shared__ unsigned int h[];
+    __shared__ Q18Stats ws[kPhThreads / 32];
+    __shared__ unsigned long long wc[kPhThreads / 32];
+    __shared__ Q18Plan s_plan;
+    const int nb = 1 << bucket_bits;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    if (big && blockIdx.x == 0 && threadIdx.x == 0) *big = 0;  // the emit's oversized-bucket list
+    for (int i = threadIdx.x; i < nb; i += kPhThreads) h[i] = 0;
+    uint64_t r0, r1;
+    ob_range(n_o, r0, r1);
+    long long amin = INT64_MAX, amax = INT64_MIN;
+    unsigned long long c = 0;
+    const uint64_t keep = l2_policy_evict_last();  // re-read by the count phase below
+    constexpr int U = 8;
+    for (uint64_t r = r0 + threadIdx.x; r < r1; r += (uint64_t)U * kPhThreads) {
+        unsigned long long ax[U], ay[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const uint64_t x = r + (uint64_t)u * kPhThreads;
+            ax[u] = ay[u] = 0;
+            if (x < r1) ld16_policy(reinterpret_cast<const ulonglong2 *>(acc + x), ax[u], ay[u], keep);
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+            const long long sum = (long long)ax[u];
+            if ((unsigned int)ay[u] > 0 && sum > having) {
+                amin = sum < amin ? sum : amin; amax = sum > amax ? sum : amax;
+                ++c;
+            }
+        }
+    }
+    amin = wmin(amin); amax = wmax(amax);
+    for (int o = 16; o; o >>= 1) c += __shfl_xor_sync(kFull, c, o);
+    if (lane == 0) { ws[warp] = Q18Stats{amin, amax, 0, 0}; wc[warp] = c; }
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        long long b0 = INT64_MAX, b1 = INT64_MIN;
+        unsigned long long bc = 0;
+        for (int k = 0; k < kPhThreads / 32; ++k) {
+            b0 = min(b0, ws[k].amt_min); b1 = max(b1, ws[k].amt_max); bc += wc[k];
+        }
+        part[blockIdx.x] = Q18Stats{b0, b1, 0, 0};
+        cpart[blockIdx.x] = bc;
+        __threadfence();
+        const unsigned long long t = atomicAdd(gbar, 1ull);
+        const unsigned long long target = (t / gridDim.x + 1) * gridDim.x;
+        // bounded wait: should the grid ever not be co-resident (another tenant on the device), a
+        // block gives up after 2 s and flags the query, which the host then redoes on the v2 path
+        unsigned long long t0;
+        asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t0));
+        while (ld_acquire_gpu_u64(gbar) < target) {
+            __nanosleep(32);
+            unsigned long long now;
+            asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(now));
+            if (now - t0 > 2000000000ull) { atomicOr(flag, kFlagHoles); break; }
+        }
+    }
+    __syncthreads();
+    if (warp == 0) {  // every block folds all partials (independent loads) and derives the plan
+        long long a0 = INT64_MAX, a1 = INT64_MIN;
+        unsigned long long cc = 0;
+        for (unsigned k = lane; k < gridDim.x; k += 32) {
+            const long long *src = reinterpret_cast<const long long *>(part + k);
+            a0 = min(a0, __ldcg(src + 0)); a1 = max(a1, __ldcg(src + 1));
+            cc += __ldcg(cpart + k);
+        }
+        a0 = wmin(a0); a1 = wmax(a1);
+        for (int o = 16; o; o >>= 1) cc += __shfl_xor_sync(kFull, cc, o);
+        if (lane == 0) {
+            const Q18Stats g{a0, a1, zone.e_min, zone.e_max};  // o_entry_d: the zone map (has_e)
+            Q18Plan P = make_q18_plan_vals(g, zone, cc, cc >= 1, bucket_bits, 1, blockIdx.x == 0 ? flag : nullptr);
+            if (cc == 0) P.spec.carry = 1;  // nothing to order: no record is ever decoded
+            // buckets must lie inside field a for the count below (else, rare: the v2 row path)
+            if (P.spec.carry && cc >= 1 && P.shift < P.spec.prefix_bits - P.spec.bits_a) P.spec.carry = 0;
+            s_plan = P;
+            if (blockIdx.x == 0) { *plan = P; *stats = g; *count = cc; }
+        }
+    }
+    __syncthreads();
+    const Q18SortSpec sp = s_plan.spec;
+    const int shift = s_plan.shift;
+    if (sp.carry && shift >= sp.prefix_bits - sp.bits_a) {  // buckets inside field a
+        const int sa = shift - (sp.prefix_bits - sp.bits_a);
+        for (uint64_t r = r0 + threadIdx.x; r < r1; r += (uint64_t)U * kPhThreads) {
+            ulonglong2 a[U];
+#pragma unroll
+            for (int u = 0; u < U; ++u) {
+                const uint64_t x = r + (uint64_t)u * kPhThreads;
+                a[u] = x < r1 ? __ldcg(reinterpret_cast<const ulonglong2 *>(acc + x)) : make_ulonglong2(0, 0);
+            }
+#pragma unroll
+            for (int u = 0; u < U; ++u) {
+                const long long sum = (long long)a[u].x;
+                if ((unsigned int)a[u].y > 0 && sum > having) {
+                    const unsigned int b = (unsigned int)(field_a(sum, sp) >> sa);
+                    H2TAP_CHECK(b < (unsigned int)nb);
+                    atomicAdd(&h[b], 1u);
+                }
+            }
+        }
+    }
+    __syncthreads();
+    unsigned int *row = mat + (uint64_t)blockIdx.x * nb;
+    for (int i = threadIdx.x; i < nb; i += kPhThreads) row[i] = h[i];
+}
+
+// Whether the fused plan + count kernel can run: its grid (ob_grid blocks) resident at once.
+bool q18_plan_hist_ok(int num_sms, int bucket_bits) {
+    int per_sm = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, q18_plan_hist_kernel, kPhThreads,
+                                                      4 << bucket_bits) != cudaSuccess) {
+        cudaGetLastError();
+        return false;
+    }
+    return (long long)per_sm * num_sms >= ob_grid(num_sms);
+}
+
+void launch_q18_plan_hist(const Q18Scratch &s, uint64_t n_o, int64_t having, unsigned long long *cpart,
+                          unsigned long long *gbar, unsigned long long *count, const Q18Zone &zone,
+                          int bucket_bits, Q18Plan *plan, unsigned int *flag, const BucketSort &bs, int num_sms,
+                          cudaStream_t st) {
+    launch_pdl(q18_plan_hist_kernel, ob_grid(num_sms), kPhThreads, 4 << bucket_bits, st, (const Q18Acc *)s.acc, n_o,
+               (long long)having, s.stat_part, cpart, gbar, s.stats, count, zone, bucket_bits, plan, flag, bs.mat,
+               bs.big);
+    count_launches(1);
+}
+
 void launch_q18_acc_stats(const Q18Scratch &s, const int64_t *o_ent, uint64_t n_o, int64_t having,
                           unsigned long long *cpart, unsigned long long *count, const Q18PlanArgs *plan_args,
                           int bucket_bits, Q18Plan *plan, unsigned int *flag, int num_sms, cudaStream_t st) {
@@ -1707,7 +1854,7 @@ void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, c
                   const int32_t *o_cnt, const int64_t *o_ent, uint64_t n_o, const int32_t *c_last,
                   int64_t having, const Q18Scratch &s, const Q18Plan *plan, int bucket_bits,
                   const BucketSort &bs, unsigned int *cnt_part, const Q18Cols &dst, unsigned int *flag,
-                  int num_sms, cudaStream_t st, PhaseMarks *marks) {
+                  int num_sms, cudaStream_t st, PhaseMarks *marks, bool counted) {
     auto begin = [&](const char *nm) { if (marks) marks->begin(nm); };
     auto end = [&] { if (marks) marks->end(); };
     const int nb = 1 << bucket_bits;
@@ -1716,12 +1863,14 @@ void q18_order_v3(const int32_t *o_w, const int32_t *o_d, const int32_t *o_id, c
     // column scan, then HAVING writes every record at its final bucket position
     const char *dx = std::getenv("H2TAP_ORDER_DIRECT");  // (read per query: tests switch it)
     const bool direct = !(dx && dx[0] == '0');
-    if (direct) {
+    if (direct || counted) {
+        if (!counted) {  // (counted: q18_plan_hist ran the count with the plan)
         begin("q18_bucket_count");
         launch_pdl(q18_acc_hist_kernel, G, kObThreads, 4 * nb, st, (const Q18Acc *)s.acc, o_w, o_d, o_id, o_ent, n_o,
                    (long long)having, plan, nb, bs.mat, bs.big);
         count_launches(1);
         end();
+        }
         begin("q18_sort_scan");
         launch_pdl(ob_scan_kernel, (nb + 31) / 32 + (kv_touch_mode() == 1 ? num_sms : 0), 32 * kScanWarps,
                    4 * std::max(32 * G, nb), st, bs.mat, G, nb, bs.count, bs.offset, bs.ticket, plan,

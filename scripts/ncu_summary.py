@@ -78,7 +78,7 @@ if traffic:
              "q1_tma_kernel<1, 0>": "q61_shared_scan", "q1_tma_kernel<1, 1>": "q6118_full_pass",
              "q18_acc_stats_kernel": "q18_acc_stats", "q18_having_rec_kernel": "q18_having_records",
              "q18_having_rec_kernel<1>": "q18_having_records", "q18_having_rec_kernel<0>": "q18_having_records",
-             "q18_acc_hist_kernel": "q18_bucket_count",
+             "q18_acc_hist_kernel": "q18_bucket_count", "q18_plan_hist_kernel": "q18_plan_count",
              "ob_scatter_rec_kernel": "q18_bucket_scatter",
              "bucket_local_emit_kernel<1536, 0, 1>": "q18_bucket_sort_emit",
              "bucket_local_emit_kernel<8192, 1536, 1>": "q18_bucket_sort_emit_large"}

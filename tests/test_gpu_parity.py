@@ -431,8 +431,10 @@ def test_profile_reports_kernels(h, eng, L):
     names = [k for k, _ in r.kernels]
     # v3 ORDER BY: bucket counts from the accumulators, the column scan, then the
     # HAVING pass writes each carry record at its final bucket position (no scatter pass)
-    assert {"q18_build", "q18_probe_groupjoin", "q18_acc_stats", "q18_bucket_count", "q18_sort_scan",
-            "q18_having_records", "q18_bucket_sort_emit"} <= set(names)
+    # (the plan and the counts in one grid-barrier kernel when the engine is alone on the device)
+    assert {"q18_build", "q18_probe_groupjoin", "q18_sort_scan", "q18_having_records",
+            "q18_bucket_sort_emit"} <= set(names)
+    assert {"q18_plan_count"} <= set(names) or {"q18_acc_stats", "q18_bucket_count"} <= set(names), names
     assert "q18_bucket_scatter" not in names
     assert all(ms >= 0 for _, ms in r.kernels) and r.device_ms > 0
     r.free()
