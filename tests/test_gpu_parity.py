@@ -905,3 +905,34 @@ def test_full_pass_batch_empty_tables(h, empty):
             assert_q18(got[2], oracle.q18(t, -100))
     finally:
         h.h2tap_close(e)
+
+
+def test_full_size_w100_full_pass_shuffled_orders(h, w100):
+    """BASELINE configs[1]/[2] size with the orders table shuffled: the bench's Q6 + Q1 + Q18 batch
+    (the full pass) then probes through the perfect-hash slot array instead of the
+    positional index, and the forced hash-join plan through open addressing — element by element
+    vs the oracle (whose result does not depend on the row order)."""
+    rng = np.random.default_rng(100)
+    t = dict(w100)
+    perm = rng.permutation(len(w100["orders"]["o_id"]))
+    t["orders"] = {k: v[perm].copy() for k, v in w100["orders"].items()}
+    e = h.h2tap_open(0)
+    try:
+        h.h2tap_load_snapshot(e, h.hot_path_tables(t), 1)
+        want6 = oracle.q6(t, Q6_D_LO, Q6_D_HI, Q6_Q_LO, Q6_Q_HI)
+        want1 = oracle.q1(t, Q1_CUTOFF)
+        want18 = oracle.q18(t, Q18_HAVING)
+        for f18 in (0, HASH):
+            rs = h.h2tap_run_queries(e, [(6, None, h.H2TAP_RESULT_DEVICE), (1, None, h.H2TAP_RESULT_DEVICE),
+                                         (18, None, h.H2TAP_RESULT_DEVICE | f18)])
+            got = []
+            for r in rs:
+                x = r.to_numpy()
+                x["_nulls"] = {k: (v.copy() if hasattr(v, "copy") else v) for k, v in r.nulls.items()}
+                got.append(x)
+                h.h2tap_free(r)
+            assert_q6(got[0], want6)
+            assert_q1(got[1], want1)
+            assert_q18(got[2], want18)
+    finally:
+        h.h2tap_close(e)
